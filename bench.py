@@ -1,0 +1,347 @@
+#!/usr/bin/env python
+"""Benchmark of the IS colouring hot path (BASELINE.json).
+
+One "step" = one complete colouring (every round of the hot path, 8(a) a0-a8)
+of a device-resident CSR graph through the C ABI (gc_color_ex).  Default
+workload at N=1: R-MAT scale 24, edge factor 16, max-min (cfg4, the config the
+BASELINE target is quoted on).  With N GPUs the graph is R-MAT scale 24+log2 N
+(weak scaling: nnz per GPU fixed; N=8 is cfg5's scale 27) partitioned by 1D
+vertex ranges.
+
+Metric: GTEPS = directed CSR entries (nnz) per colouring / device time, the
+whole job's throughput.  Timing: W warm-up colourings, then K colourings each
+bracketed by CUDA events on the launching stream, L2 flushed (256 MiB write)
+before each one outside the events; barrier + synchronize around the timed
+region; max over ranks.
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--impl gc|reference]
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import math
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+METRIC = "GTEPS (directed CSR entries / device ms per colouring)"
+UNIT = "GTEPS"
+
+
+def parse():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=10)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--impl", default="gc", choices=["gc", "reference"])
+    ap.add_argument("--scale", type=int, default=0, help="R-MAT scale (default 24+log2 N)")
+    ap.add_argument("--variant", default="maxmin", choices=["maxmin", "luby", "multihash"])
+    ap.add_argument("--hashes", type=int, default=4)
+    ap.add_argument("--mode", default="auto", choices=["auto", "sweep", "event"])
+    ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--no-profile", action="store_true")
+    ap.add_argument("--cpu-scale", type=int, default=20, help="R-MAT scale of the oracle sample")
+    ap.add_argument("--quiet", action="store_true")
+    return ap.parse_args()
+
+
+def env_rank():
+    return (int(os.environ.get("RANK", 0)), int(os.environ.get("WORLD_SIZE", 1)),
+            int(os.environ.get("LOCAL_RANK", 0)))
+
+
+def log(*a):
+    print(*a, file=sys.stderr, flush=True)
+
+
+# ------------------------------------------------------------------ clocks
+class ClockSampler:
+    """nvidia-smi sampling DURING the timed region (B200_PROFILING.md)."""
+
+    FIELDS = ("clocks.sm,clocks.max.sm,power.draw,clocks_event_reasons.hw_slowdown,"
+              "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
+              "clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, index: int):
+        self.index = index
+        self.proc = None
+        self.lines = []
+
+    def start(self):
+        try:
+            self.proc = subprocess.Popen(
+                ["nvidia-smi", "-i", str(self.index), f"--query-gpu={self.FIELDS}",
+                 "--format=csv,noheader,nounits", "-lms", "100"],
+                stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+            threading.Thread(target=self._read, daemon=True).start()
+        except Exception:
+            self.proc = None
+
+    def _read(self):
+        for line in self.proc.stdout:
+            self.lines.append(line.strip())
+
+    def stop(self):
+        if self.proc:
+            time.sleep(0.25)
+            self.proc.terminate()
+            try:
+                self.proc.wait(timeout=2)
+            except Exception:
+                self.proc.kill()
+        sm, mx, reasons = [], [], set()
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        for ln in self.lines:
+            parts = [p.strip() for p in ln.split(",")]
+            if len(parts) < 7:
+                continue
+            try:
+                sm.append(float(parts[0]))
+                mx.append(float(parts[1]))
+            except ValueError:
+                continue
+            for nm, val in zip(names, parts[3:7]):
+                if val.lower().startswith("active"):
+                    reasons.add(nm)
+        if not sm:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": [], "samples": 0}
+        return {"sm_mhz": statistics.median(sm), "sm_max_mhz": max(mx),
+                "reasons": sorted(reasons), "samples": len(sm)}
+
+
+def measured_peaks():
+    try:
+        with open(os.path.join(ROOT, "MEASURED_PEAKS.json")) as f:
+            p = json.load(f)
+        return float(p["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs)"
+    except Exception:
+        return 6650.0, "fallback (B200_PROFILING.md 6.65 TB/s)"
+
+
+def ncu_traffic(workload: str):
+    """Per-launch DRAM bytes of the dominant kernel from a committed ncu
+    --set full capture (profiles/ncu_traffic.json), or None."""
+    try:
+        with open(os.path.join(ROOT, "profiles", "ncu_traffic.json")) as f:
+            d = json.load(f)
+        ent = d.get(workload)
+        return None if ent is None else ent.get("dram_bytes_per_launch")
+    except Exception:
+        return None
+
+
+# --------------------------------------------------------------- reference
+def cpu_sample(scale: int, variant: str, hashes: int):
+    """The oracle as it stands, on a bounded sample of the workload: a full
+    colouring of the same generator at a smaller scale.  Returns dict."""
+    import graphgen as G
+    import oracle as O
+    g = G.rmat(scale, 16, seed=1)
+    O.lib()
+    t0 = time.perf_counter()
+    if variant == "luby":
+        O.color_luby(g, 1)
+    else:
+        O.color_maxmin(g, 1, hashes if variant == "multihash" else 1)
+    dt = time.perf_counter() - t0
+    return {"value": g.nnz / dt / 1e9, "unit": UNIT, "cores": O.num_threads(), "kind": "oracle",
+            "sample": f"one full {variant} colouring of R-MAT scale {scale} ef16 (nnz {g.nnz}) "
+                      f"by oracle/oracle.c with OpenMP; {dt:.2f} s",
+            "seconds": dt}
+
+
+def run_reference(args, rank, world):
+    if rank != 0:
+        return
+    import graphgen as G
+    import oracle as O
+    scale = max(10, args.cpu_scale - 1)
+    g = G.rmat(scale, 16, seed=1)
+    O.lib()
+    times = []
+    for i in range(args.warmup + args.steps):
+        t0 = time.perf_counter()
+        if args.variant == "luby":
+            O.color_luby(g, 1)
+        else:
+            O.color_maxmin(g, 1, args.hashes if args.variant == "multihash" else 1)
+        dt = time.perf_counter() - t0
+        if i >= args.warmup:
+            times.append(dt)
+    total = sum(times)
+    value = g.nnz * len(times) / total / 1e9
+    line = {"impl": "reference", "metric": METRIC, "value": value, "unit": UNIT,
+            "n_gpus": args.gpus, "steps": args.steps, "warmup": args.warmup,
+            "ms_per_step": 1e3 * total / len(times), "higher_is_better": True,
+            "scaling": "weak", "vs_baseline": None, "dtype": "u32", "data": "synthetic",
+            "config": {"workload": f"rmat-s{scale}-ef16 {args.variant} (bounded CPU sample of "
+                                   f"the bench workload)", "variant": args.variant, "seed": 1,
+                       "n": g.n, "nnz": g.nnz, "parallelism": "OpenMP host threads"},
+            "cpu_baseline": {"value": value, "unit": UNIT, "cores": O.num_threads(),
+                             "kind": "oracle",
+                             "sample": f"each step: one full colouring of R-MAT scale {scale}"},
+            "e2e": {"value": value, "unit": UNIT, "h2d_bytes_per_step": 0,
+                    "d2h_bytes_per_step": 0}}
+    print(json.dumps(line), flush=True)
+
+
+# -------------------------------------------------------------------- main
+def main():
+    args = parse()
+    rank, world, local = env_rank()
+    if args.impl == "reference":
+        run_reference(args, rank, world)
+        return
+    import torch
+    import torch.distributed as dist
+
+    import graphgen as G
+    import paper_conf_ipps_osamatybo19_b200 as gcb
+
+    torch.cuda.set_device(local)
+    dev = torch.device("cuda", local)
+    if world > 1:
+        dist.init_process_group("nccl", device_id=dev)
+    scale = args.scale or (24 + int(round(math.log2(max(1, world)))))
+    variant = {"maxmin": gcb.MAXMIN, "luby": gcb.LUBY_MIS,
+               "multihash": gcb.MULTIHASH(args.hashes)}[args.variant]
+    mode = {"auto": gcb.MODE_AUTO, "sweep": gcb.MODE_SWEEP, "event": gcb.MODE_EVENT}[args.mode]
+
+    t0 = time.time()
+    if world > 1:
+        from paper_conf_ipps_osamatybo19_b200 import dist as gdist
+        g, handle, n, nnz_global = gdist.build_partitioned_rmat(scale, 16, 1, rank, world, dev)
+    else:
+        g = G.rmat(scale, 16, seed=1, device=dev)
+        n, nnz_global = g.n, g.nnz
+        handle = gcb.Graph(g.n, g.row_offsets, g.col_indices, flags=gcb.BORROW_DEVICE)
+    torch.cuda.synchronize()
+    if rank == 0 and not args.quiet:
+        log(f"graph rmat s{scale}: n={n} nnz={nnz_global} built in {time.time() - t0:.1f}s")
+    stream = torch.cuda.current_stream()
+    handle.set_stream(stream)
+    out = torch.empty(n, dtype=torch.int32, device=dev)
+    flush = torch.empty(256 << 20, dtype=torch.uint8, device=dev)
+
+    def barrier():
+        if world > 1:
+            dist.barrier()
+
+    kw = dict(mode=mode, stats=True)
+    for _ in range(args.warmup):
+        _, ncol, st = handle.color(1, variant, out, **kw)
+    torch.cuda.synchronize()
+    barrier()
+
+    clocks = ClockSampler(local)
+    clocks.start()
+    ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True))
+          for _ in range(args.steps)]
+    launches = 0
+    rounds = []
+    barrier()
+    torch.cuda.synchronize()
+    for i in range(args.steps):
+        flush.fill_(i & 0xFF)          # L2 flush, outside the timed events
+        ev[i][0].record(stream)
+        _, ncol, st = handle.color(1, variant, out, **kw)
+        ev[i][1].record(stream)
+        launches += st.launches
+        rounds.append(st.rounds)
+    torch.cuda.synchronize()
+    barrier()
+    clk = clocks.stop()
+    step_ms = [a.elapsed_time(b) for a, b in ev]
+    total_ms = sum(step_ms)
+    if world > 1:
+        t = torch.tensor([total_ms], dtype=torch.float64, device=dev)
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        total_ms = float(t.item())
+    ms_per = total_ms / args.steps
+    value = nnz_global * args.steps / (total_ms / 1e3) / 1e9
+    mode_used = {1: "sweep", 2: "event"}.get(st.mode_used, str(st.mode_used))
+
+    # ---- roofline of the dominant kernel: a profiled pass (GC_PROFILE brackets
+    # every sweep launch with events on this stream); separate from the timed steps
+    roof = None
+    if not args.no_profile:
+        _, _, sp = handle.color(1, variant, out, flags=gcb.PROFILE, **kw)
+        torch.cuda.synchronize()
+        peak, peak_src = measured_peaks()
+        cls = max(range(4), key=lambda c: sp.kernel_ms[c])
+        name = {0: "sweep", 1: "hub", 2: "other", 3: "other"}[cls]
+        kms, kl, kb = sp.kernel_ms[cls], sp.kernel_launches[cls], sp.kernel_bytes[cls]
+        achieved = (kb / 1e9) / (kms / 1e3) if kms > 0 else 0.0
+        roof = {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
+                "frac": achieved / peak, "traffic": ncu_traffic(f"rmat-s{scale}-{args.variant}"),
+                "kernel": name, "launches": kl, "avg_launch_us": 1e3 * kms / max(kl, 1),
+                "bytes_per_launch": kb / max(kl, 1), "kernel_share_of_step":
+                kms / max(sp.ms, 1e-9), "peak_source": peak_src,
+                "visits": sp.visits, "profiled_ms": sp.ms}
+
+    # ---- end to end through the C ABI with host buffers
+    e2e = None
+    if not args.no_e2e and world == 1:
+        ro_h = g.row_offsets.cpu().pin_memory()
+        ci_h = g.col_indices.cpu().pin_memory()
+        out_h = torch.empty(n, dtype=torch.int32).pin_memory()
+        dstream = torch.cuda.default_stream()
+        e2e_ms = []
+        for i in range(max(1, min(args.steps, 5)) + 1):
+            flush.fill_(i & 0xFF)
+            torch.cuda.synchronize()
+            a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            a.record(dstream)
+            with gcb.Graph(n, ro_h, ci_h) as h2:
+                h2.color(1, variant, out_h, mode=mode)
+            b.record(dstream)
+            torch.cuda.synchronize()
+            if i > 0:  # first call warms allocations
+                e2e_ms.append(a.elapsed_time(b))
+        em = sum(e2e_ms) / len(e2e_ms)
+        e2e = {"value": nnz_global / (em / 1e3) / 1e9, "unit": UNIT,
+               "h2d_bytes_per_step": 8 * (n + 1) + 4 * nnz_global,
+               "d2h_bytes_per_step": 4 * n, "ms_per_step": em,
+               "includes": "gc_create_csr (H2D copy + validation) + gc_color (D2H colours) + "
+                           "gc_destroy, pinned host buffers"}
+
+    cpu = None
+    if rank == 0 and world == 1 and not args.no_cpu_baseline:
+        cpu = cpu_sample(args.cpu_scale, args.variant, args.hashes)
+
+    if rank == 0:
+        line = {"metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world,
+                "steps": args.steps, "warmup": args.warmup, "ms_per_step": ms_per,
+                "higher_is_better": True, "scaling": "weak", "vs_baseline": None,
+                "dtype": "u32", "data": "synthetic",
+                "config": {"workload": f"rmat-s{scale}-ef16 {args.variant}"
+                                       + (f" H={args.hashes}" if args.variant == "multihash" else "")
+                                       + (" (cfg4)" if scale == 24 else
+                                          " (cfg5)" if scale == 27 else ""),
+                           "generator": "Graph500 Kronecker A,B,C=.57,.19,.19, symmetrised, "
+                                        "seeded label permutation, graph seed 1",
+                           "n": n, "nnz": nnz_global, "variant": args.variant, "seed": 1,
+                           "mode": mode_used,
+                           "parallelism": "1 GPU" if world == 1 else f"1D vertex ranges x{world}",
+                           "l2": "flushed before every timed colouring (256 MiB write outside "
+                                 "the events); col_indices alone exceed L2"},
+                "n_colors": ncol, "rounds": rounds[-1],
+                "ms_per_step_median": statistics.median(step_ms),
+                "clocks": clk, "gpu_launches": launches,
+                "roofline": roof, "cpu_baseline": cpu, "e2e": e2e}
+        print(json.dumps(line), flush=True)
+    handle.close()
+    if world > 1:
+        dist.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

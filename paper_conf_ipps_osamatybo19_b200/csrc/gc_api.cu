@@ -1,0 +1,614 @@
+// gc_api.cu -- the C ABI declared in include/gc.h: handle lifecycle, input
+// validation, variant dispatch, output and colour counting.
+#include <algorithm>
+#include <cstdio>
+#include <cstring>
+#include <new>
+#include <string>
+
+#include "gc_internal.cuh"
+
+namespace gc {
+
+static thread_local std::string g_last_error;
+
+void set_error(const std::string &msg) { g_last_error = msg; }
+
+int cuda_fail(cudaError_t e, const char *what) {
+    char buf[512];
+    snprintf(buf, sizeof(buf), "CUDA error %s (%s) in %s", cudaGetErrorName(e),
+             cudaGetErrorString(e), what);
+    set_error(buf);
+    cudaGetLastError();  // clear sticky-free errors
+    return e == cudaErrorMemoryAllocation ? GC_ERR_OOM : GC_ERR_CUDA;
+}
+
+bool is_device_ptr(const void *p) {
+    if (!p) return false;
+    cudaPointerAttributes a;
+    if (cudaPointerGetAttributes(&a, p) != cudaSuccess) {
+        cudaGetLastError();
+        return false;
+    }
+    return a.type == cudaMemoryTypeDevice || a.type == cudaMemoryTypeManaged;
+}
+
+namespace {
+
+constexpr int kCtrWords = 64;
+
+__global__ void k_validate(const int64_t *__restrict__ ro, const uint32_t *__restrict__ ci,
+                           int64_t n, int64_t nnz, int64_t n_global, int64_t v_begin,
+                           unsigned long long *err) {
+    // err[0]: non-monotone / out-of-range offsets; err[1]: col >= n; err[2]: self-loop;
+    // err[3]: max degree
+    for (int64_t v = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; v < n;
+         v += (int64_t)gridDim.x * blockDim.x) {
+        int64_t a = ro[v], b = ro[v + 1];
+        if (a > b || a < 0 || b > nnz) {
+            atomicAdd(&err[0], 1ull);
+            continue;
+        }
+        atomicMax(&err[3], (unsigned long long)(b - a));
+        for (int64_t e = a; e < b; ++e) {
+            uint32_t u = ci[e];
+            if ((int64_t)u >= n_global) atomicAdd(&err[1], 1ull);
+            else if ((int64_t)u == v + v_begin) atomicAdd(&err[2], 1ull);
+        }
+    }
+}
+
+// Symmetry: for every entry (v,u) some entry (u,v) exists.  Linear scan of
+// row u (rows may be unsorted); O(sum deg^2) worst case, opt-in only.
+__global__ void k_validate_sym(const int64_t *__restrict__ ro, const uint32_t *__restrict__ ci,
+                               int64_t n, unsigned long long *err) {
+    const int lane = threadIdx.x & 31;
+    const int64_t warp = ((int64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+    const int64_t nwarps = ((int64_t)gridDim.x * blockDim.x) >> 5;
+    for (int64_t v = warp; v < n; v += nwarps) {
+        for (int64_t e = ro[v]; e < ro[v + 1]; ++e) {
+            uint32_t u = ci[e];
+            bool found = false;
+            for (int64_t f0 = ro[u]; f0 < ro[u + 1]; f0 += 32) {
+                int64_t f = f0 + lane;
+                bool hit = f < ro[u + 1] && ci[f] == (uint32_t)v;
+                if (__any_sync(0xFFFFFFFFu, hit)) {
+                    found = true;
+                    break;
+                }
+            }
+            if (!found && lane == 0) atomicAdd(&err[4], 1ull);
+        }
+    }
+}
+
+__global__ void k_priorities(uint64_t v_begin, int64_t count, uint32_t key, uint32_t *out) {
+    for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < count;
+         i += (int64_t)gridDim.x * blockDim.x)
+        out[i] = weight_mix((uint32_t)(v_begin + (uint64_t)i) ^ key);
+}
+
+__global__ void k_max_u32(const uint32_t *__restrict__ C, int64_t n, unsigned long long *mx) {
+    uint32_t m = 0;
+    for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n;
+         i += (int64_t)gridDim.x * blockDim.x)
+        m = max(m, C[i]);
+    m = __reduce_max_sync(0xFFFFFFFFu, m);
+    if ((threadIdx.x & 31) == 0) atomicMax(mx, (unsigned long long)m);
+}
+
+__global__ void k_mark(const uint32_t *__restrict__ C, int64_t n, uint32_t *bitmap) {
+    for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n;
+         i += (int64_t)gridDim.x * blockDim.x) {
+        uint32_t c = C[i];
+        uint32_t bit = 1u << (c & 31);
+        if (!(bitmap[c >> 5] & bit)) atomicOr(&bitmap[c >> 5], bit);
+    }
+}
+
+__global__ void k_popc(const uint32_t *__restrict__ bitmap, int64_t words, unsigned long long *cnt) {
+    unsigned long long s = 0;
+    for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < words;
+         i += (int64_t)gridDim.x * blockDim.x)
+        s += __popc(bitmap[i]);
+    s = __reduce_add_sync(0xFFFFFFFFu, (unsigned)s);
+    if ((threadIdx.x & 31) == 0 && s) atomicAdd(cnt, s);
+}
+
+// Exclusive prefix of popcounts over the bitmap words (single CTA; the
+// bitmap has <= 2^27 words so this loops in chunks), then rank lookup.
+__global__ void k_rank_words(const uint32_t *__restrict__ bitmap, int64_t words, uint32_t *rank) {
+    __shared__ uint32_t carry;
+    __shared__ uint32_t warp_sums[32];
+    if (threadIdx.x == 0) carry = 0;
+    __syncthreads();
+    for (int64_t base = 0; base < words; base += blockDim.x) {
+        int64_t i = base + threadIdx.x;
+        uint32_t x = i < words ? (uint32_t)__popc(bitmap[i]) : 0u;
+        // inclusive warp scan
+        uint32_t y = x;
+        for (int d = 1; d < 32; d <<= 1) {
+            uint32_t z = __shfl_up_sync(0xFFFFFFFFu, y, d);
+            if ((threadIdx.x & 31) >= d) y += z;
+        }
+        if ((threadIdx.x & 31) == 31) warp_sums[threadIdx.x >> 5] = y;
+        __syncthreads();
+        if (threadIdx.x < 32) {
+            uint32_t w = threadIdx.x < (blockDim.x >> 5) ? warp_sums[threadIdx.x] : 0u;
+            uint32_t ws = w;
+            for (int d = 1; d < 32; d <<= 1) {
+                uint32_t z = __shfl_up_sync(0xFFFFFFFFu, ws, d);
+                if (threadIdx.x >= d) ws += z;
+            }
+            warp_sums[threadIdx.x] = ws - w;  // exclusive
+        }
+        __syncthreads();
+        uint32_t excl = carry + warp_sums[threadIdx.x >> 5] + (y - x);
+        if (i < words) rank[i] = excl;
+        __syncthreads();
+        if (threadIdx.x == blockDim.x - 1) carry = excl + x;
+        __syncthreads();
+    }
+}
+
+__global__ void k_remap(uint32_t *C, int64_t n, const uint32_t *__restrict__ bitmap,
+                        const uint32_t *__restrict__ rank) {
+    for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n;
+         i += (int64_t)gridDim.x * blockDim.x) {
+        uint32_t c = C[i];
+        uint32_t w = c >> 5, b = c & 31;
+        C[i] = rank[w] + (uint32_t)__popc(bitmap[w] & ((1u << b) - 1u));
+    }
+}
+
+int grid_for(int64_t n, int sm) {
+    return (int)std::max<int64_t>(1, std::min<int64_t>((n + 255) / 256, (int64_t)sm * 8));
+}
+
+int current_device_ok(int *dev, int *sms) {
+    int count = 0;
+    cudaError_t e = cudaGetDeviceCount(&count);
+    if (e != cudaSuccess || count == 0) {
+        cudaGetLastError();
+        set_error("no CUDA device available (libgc has no CPU fallback)");
+        return GC_ERR_CUDA;
+    }
+    GC_CUDA_TRY(cudaGetDevice(dev));
+    GC_CUDA_TRY(cudaDeviceGetAttribute(sms, cudaDevAttrMultiProcessorCount, *dev));
+    int major = 0;
+    GC_CUDA_TRY(cudaDeviceGetAttribute(&major, cudaDevAttrComputeCapabilityMajor, *dev));
+    if (major < 10) {
+        set_error("libgc is built for sm_100a (Blackwell B200); this device is older");
+        return GC_ERR_CUDA;
+    }
+    return GC_OK;
+}
+
+}  // namespace
+
+int fill_u32(uint32_t *p, uint32_t val, int64_t n, cudaStream_t st);
+
+int ensure_nk(gc_graph *g, int64_t need) {
+    Scratch &s = g->s;
+    if (need <= s.nk_cap) return GC_OK;
+    int64_t cap = std::max<int64_t>(need * 2, 1 << 12);
+    int64_t *nk = nullptr;
+    GC_CUDA_TRY(cudaMalloc(&nk, sizeof(int64_t) * cap));
+    if (s.nk) {
+        GC_CUDA_TRY(cudaMemcpyAsync(nk, s.nk, sizeof(int64_t) * s.nk_cap, cudaMemcpyDeviceToDevice,
+                                    g->stream));
+        GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
+        cudaFree(s.nk);
+    }
+    s.nk = nk;
+    s.nk_cap = cap;
+    return GC_OK;
+}
+
+int ensure_scratch(gc_graph *g, bool need_event, bool need_luby) {
+    Scratch &s = g->s;
+    const size_t nn = (size_t)std::max<int64_t>(g->n, 1);
+    if (!s.C) {
+        GC_CUDA_TRY(cudaMalloc(&s.C, nn * 4));
+        GC_CUDA_TRY(cudaMalloc(&s.F[0], nn * 4));
+        GC_CUDA_TRY(cudaMalloc(&s.F[1], nn * 4));
+        GC_CUDA_TRY(cudaMalloc(&s.hub, nn * 4));
+        GC_CUDA_TRY(cudaMalloc(&s.ctr, kCtrWords * sizeof(unsigned long long)));
+        GC_CUDA_TRY(cudaMemset(s.ctr, 0, kCtrWords * sizeof(unsigned long long)));
+        GC_CUDA_TRY(cudaMallocHost(&s.host_pinned, 4096));
+        int rc = ensure_nk(g, 1 << 12);
+        if (rc) return rc;
+    }
+    if ((need_luby || need_event) && !s.S) GC_CUDA_TRY(cudaMalloc(&s.S, nn * 4));
+    if (need_event && !s.W) {
+        GC_CUDA_TRY(cudaMalloc(&s.W, nn * 8));
+        GC_CUDA_TRY(cudaMalloc(&s.P, nn * 8));
+    }
+    return GC_OK;
+}
+
+// Distinct colours of C[0..n); optionally renumber in place (R12).
+int64_t count_colors_device(gc_graph *g, const uint32_t *C, int64_t n, bool compact,
+                            uint32_t *C_inout, int64_t *launches) {
+    if (n == 0) return 0;
+    Scratch &s = g->s;
+    cudaStream_t st = g->stream;
+    unsigned long long *tmp = s.ctr + 48;
+    GC_CUDA_TRY(cudaMemsetAsync(tmp, 0, 2 * sizeof(unsigned long long), st));
+    const int grid = grid_for(n, g->sm_count);
+    k_max_u32<<<grid, 256, 0, st>>>(C, n, tmp);
+    GC_CUDA_TRY(cudaMemcpyAsync(s.host_pinned, tmp, sizeof(unsigned long long),
+                                cudaMemcpyDeviceToHost, st));
+    GC_CUDA_TRY(cudaStreamSynchronize(st));
+    const uint64_t maxc = *reinterpret_cast<unsigned long long *>(s.host_pinned);
+    if (maxc == GC_UNC) {
+        set_error("internal: uncoloured vertex in the result");
+        return GC_ERR_CUDA;
+    }
+    const int64_t words = (int64_t)(maxc >> 5) + 1;
+    if (words > s.bitmap_words) {
+        if (s.bitmap) cudaFree(s.bitmap);
+        s.bitmap = nullptr;
+        GC_CUDA_TRY(cudaMalloc(&s.bitmap, (size_t)words * 8));  // bitmap + rank table
+        s.bitmap_words = words;
+    }
+    uint32_t *rank = s.bitmap + words;
+    GC_CUDA_TRY(cudaMemsetAsync(s.bitmap, 0, (size_t)words * 4, st));
+    k_mark<<<grid, 256, 0, st>>>(C, n, s.bitmap);
+    k_popc<<<grid_for(words, g->sm_count), 256, 0, st>>>(s.bitmap, words, tmp + 1);
+    *launches += 3;
+    if (compact) {
+        k_rank_words<<<1, 1024, 0, st>>>(s.bitmap, words, rank);
+        k_remap<<<grid, 256, 0, st>>>(C_inout, n, s.bitmap, rank);
+        *launches += 2;
+    }
+    GC_CUDA_TRY(cudaGetLastError());
+    GC_CUDA_TRY(cudaMemcpyAsync(s.host_pinned, tmp + 1, sizeof(unsigned long long),
+                                cudaMemcpyDeviceToHost, st));
+    GC_CUDA_TRY(cudaStreamSynchronize(st));
+    return (int64_t)*reinterpret_cast<unsigned long long *>(s.host_pinned);
+}
+
+int launch_priorities(uint64_t seed, int j, int64_t v_begin, int64_t count, uint32_t *out,
+                      cudaStream_t st) {
+    if (count <= 0) return GC_OK;
+    k_priorities<<<grid_for(count, 148), 256, 0, st>>>((uint64_t)v_begin, count,
+                                                      weight_key(seed, j), out);
+    GC_CUDA_TRY(cudaGetLastError());
+    return GC_OK;
+}
+
+static void free_scratch(Scratch &s) {
+    cudaFree(s.C);
+    cudaFree(s.F[0]);
+    cudaFree(s.F[1]);
+    cudaFree(s.hub);
+    cudaFree(s.S);
+    cudaFree(s.W);
+    cudaFree(s.P);
+    cudaFree(s.ctr);
+    cudaFree(s.nk);
+    cudaFree(s.bitmap);
+    if (s.host_pinned) cudaFreeHost(s.host_pinned);
+    s = Scratch();
+}
+
+void destroy_dist(gc_graph *g);  // gc_dist.cu
+
+}  // namespace gc
+
+using namespace gc;
+
+extern "C" {
+
+const char *gc_last_error(void) { return g_last_error.c_str(); }
+
+const char *gc_version(void) {
+    static char buf[64];
+    if (!buf[0]) snprintf(buf, sizeof(buf), "gc %d sm_100a cudart %d", GC_ABI_VERSION, CUDART_VERSION);
+    return buf;
+}
+
+static int create_common(int64_t n, int64_t nnz, const int64_t *row_offsets,
+                         const uint32_t *col_indices, uint32_t flags, gc_graph **out,
+                         int64_t v_begin, int64_t n_global) {
+    if (!out) {
+        set_error("gc_create_csr: out is NULL");
+        return GC_ERR_INVALID_ARG;
+    }
+    *out = nullptr;
+    if (n < 0 || nnz < 0 || !row_offsets || (nnz > 0 && !col_indices)) {
+        set_error("gc_create_csr: bad sizes or NULL arrays");
+        return GC_ERR_INVALID_ARG;
+    }
+    if (n_global >= (int64_t)1 << 32) {
+        set_error("gc_create_csr: n must be < 2^32 (uint32 vertex ids)");
+        return GC_ERR_TOO_LARGE;
+    }
+    int dev = 0, sms = 148;
+    int rc = current_device_ok(&dev, &sms);
+    if (rc) return rc;
+    gc_graph *g = new (std::nothrow) gc_graph();
+    if (!g) return GC_ERR_OOM;
+    g->device = dev;
+    g->sm_count = sms;
+    g->n = n;
+    g->n_global = n_global;
+    g->v_begin = v_begin;
+    g->nnz = nnz;
+    const bool ro_dev = is_device_ptr(row_offsets);
+    const bool ci_dev = nnz == 0 || is_device_ptr(col_indices);
+    auto fail = [&](int code) {
+        if (g->owns_csr) {
+            cudaFree(g->ro);
+            cudaFree(g->ci);
+        }
+        free_scratch(g->s);
+        delete g;
+        return code;
+    };
+    if ((flags & GC_BORROW_DEVICE) && ro_dev && ci_dev) {
+        g->owns_csr = false;
+        g->ro = const_cast<int64_t *>(row_offsets);
+        g->ci = const_cast<uint32_t *>(col_indices);
+    } else {
+        cudaError_t e = cudaMalloc(&g->ro, sizeof(int64_t) * (size_t)(n + 1));
+        if (e == cudaSuccess) e = cudaMalloc(&g->ci, sizeof(uint32_t) * (size_t)std::max<int64_t>(nnz, 1));
+        if (e != cudaSuccess) return fail(cuda_fail(e, "cudaMalloc(csr)"));
+        e = cudaMemcpy(g->ro, row_offsets, sizeof(int64_t) * (size_t)(n + 1), cudaMemcpyDefault);
+        if (e == cudaSuccess && nnz > 0)
+            e = cudaMemcpy(g->ci, col_indices, sizeof(uint32_t) * (size_t)nnz, cudaMemcpyDefault);
+        if (e != cudaSuccess) return fail(cuda_fail(e, "cudaMemcpy(csr)"));
+    }
+    // validation on the device
+    rc = ensure_scratch(g, false, false);
+    if (rc) return fail(rc);
+    int64_t first = 0, last = 0;
+    cudaError_t e = cudaMemcpy(&first, g->ro, sizeof(int64_t), cudaMemcpyDeviceToHost);
+    if (e == cudaSuccess)
+        e = cudaMemcpy(&last, g->ro + n, sizeof(int64_t), cudaMemcpyDeviceToHost);
+    if (e != cudaSuccess) return fail(cuda_fail(e, "cudaMemcpy(offsets)"));
+    if (first != 0 || last != nnz) {
+        set_error("gc_create_csr: row_offsets[0] must be 0 and row_offsets[n] == nnz");
+        return fail(GC_ERR_INVALID_ARG);
+    }
+    unsigned long long *err = g->s.ctr + 40;
+    e = cudaMemset(err, 0, 8 * sizeof(unsigned long long));
+    if (e != cudaSuccess) return fail(cuda_fail(e, "cudaMemset"));
+    if (n > 0) {
+        // the distributed path checks col < n_global (ghost ids are global)
+        k_validate<<<grid_for(n, sms), 256>>>(g->ro, g->ci, n, nnz, n_global, v_begin, err);
+        if ((flags & GC_VALIDATE) && n == n_global)
+            k_validate_sym<<<grid_for(n * 32, sms), 256>>>(g->ro, g->ci, n, err);
+    }
+    unsigned long long herr[8] = {0};
+    e = cudaMemcpy(herr, err, sizeof(herr), cudaMemcpyDeviceToHost);
+    if (e != cudaSuccess) return fail(cuda_fail(e, "validate"));
+    if (herr[0]) {
+        set_error("gc_create_csr: row_offsets are not monotone / in range");
+        return fail(GC_ERR_INVALID_ARG);
+    }
+    if (herr[1]) {
+        set_error("gc_create_csr: column index >= n");
+        return fail(GC_ERR_INVALID_ARG);
+    }
+    if (herr[2]) {
+        set_error("gc_create_csr: self-loop (never terminates; R7)");
+        return fail(GC_ERR_SELF_LOOP);
+    }
+    if (herr[4]) {
+        set_error("gc_create_csr: adjacency is not symmetric");
+        return fail(GC_ERR_NOT_SYMMETRIC);
+    }
+    g->max_deg = (int64_t)herr[3];
+    *out = g;
+    return GC_OK;
+}
+
+int gc_create_csr(int64_t n, int64_t nnz, const int64_t *row_offsets, const uint32_t *col_indices,
+                  uint32_t flags, gc_graph **out) {
+    return create_common(n, nnz, row_offsets, col_indices, flags, out, 0, n);
+}
+
+int gc_set_stream(gc_graph *g, void *cuda_stream) {
+    if (!g) {
+        set_error("gc_set_stream: NULL handle");
+        return GC_ERR_INVALID_ARG;
+    }
+    g->stream = (cudaStream_t)cuda_stream;
+    return GC_OK;
+}
+
+void gc_destroy(gc_graph *g) {
+    if (!g) return;
+    cudaSetDevice(g->device);
+    destroy_dist(g);
+    if (g->owns_csr) {
+        cudaFree(g->ro);
+        cudaFree(g->ci);
+    }
+    free_scratch(g->s);
+    delete g;
+}
+
+int64_t gc_color_dist(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_stats *stats);
+
+int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_stats *stats) {
+    if (!g || !o || o->struct_size < sizeof(gc_options)) {
+        set_error("gc_color_ex: NULL handle/options or options.struct_size too small");
+        return GC_ERR_INVALID_ARG;
+    }
+    if (g->n > 0 && !colors_out) {
+        set_error("gc_color_ex: colors_out is NULL");
+        return GC_ERR_INVALID_ARG;
+    }
+    if (stats && stats->struct_size < sizeof(gc_stats)) {
+        set_error("gc_color_ex: stats.struct_size too small");
+        return GC_ERR_INVALID_ARG;
+    }
+    const int kind = GC_VARIANT_KIND(o->variant);
+    int H = 1;
+    if (kind == GC_MULTIHASH(0)) {
+        H = GC_VARIANT_HASHES(o->variant);
+        if (H < 1 || H > GC_MAX_HASHES) {
+            set_error("gc_color_ex: multi-hash needs 1 <= h <= 16");
+            return GC_ERR_INVALID_ARG;
+        }
+    } else if (kind != GC_MAXMIN && kind != GC_LUBY_MIS) {
+        set_error("gc_color_ex: unknown variant");
+        return GC_ERR_INVALID_ARG;
+    }
+    if (o->mode < GC_MODE_AUTO || o->mode > GC_MODE_EVENT) {
+        set_error("gc_color_ex: unknown mode");
+        return GC_ERR_INVALID_ARG;
+    }
+    GC_CUDA_TRY(cudaSetDevice(g->device));
+    if (g->dist) return gc_color_dist(g, o, colors_out, stats);
+
+    const bool luby = kind == GC_LUBY_MIS;
+    int mode = o->mode;
+    if (mode == GC_MODE_AUTO) mode = GC_MODE_SWEEP;
+    if (luby) mode = GC_MODE_SWEEP;
+    if (mode == GC_MODE_EVENT && H != 1) mode = GC_MODE_SWEEP;
+
+    int rc = ensure_scratch(g, mode == GC_MODE_EVENT, luby);
+    if (rc) return rc;
+    RunParams p;
+    p.H = H;
+    for (int j = 0; j < H; ++j) p.keys.k[j] = weight_key(o->seed, j);
+    p.thread_deg_max = o->thread_deg_max > 0 ? o->thread_deg_max : 8;
+    p.hub_deg_min = o->hub_deg_min > 0 ? o->hub_deg_min : 4096;
+    p.batch_rounds = o->batch_rounds;
+    p.max_rounds = (int64_t)(0x7FFFFFFFll / (2 * H)) + 1;
+    Profile prof;
+    prof.on = (o->flags & GC_PROFILE) != 0;
+    p.prof = &prof;
+
+    cudaEvent_t e0, e1;
+    GC_CUDA_TRY(cudaEventCreate(&e0));
+    GC_CUDA_TRY(cudaEventCreate(&e1));
+    GC_CUDA_TRY(cudaEventRecord(e0, g->stream));
+    RunResult res;
+    if (luby)
+        rc = run_luby(g, p, &res);
+    else if (mode == GC_MODE_EVENT)
+        rc = run_event_maxmin(g, p, &res);
+    else
+        rc = run_sweep_maxmin(g, p, &res);
+    if (rc) {
+        cudaEventDestroy(e0);
+        cudaEventDestroy(e1);
+        return rc;
+    }
+    int64_t launches = res.launches;
+    int64_t ncol = count_colors_device(g, g->s.C, g->n, (o->flags & GC_COMPACT) != 0, g->s.C,
+                                       &launches);
+    if (ncol < 0) return ncol;
+    if (g->n > 0) {
+        GC_CUDA_TRY(cudaMemcpyAsync(colors_out, g->s.C, sizeof(int32_t) * (size_t)g->n,
+                                    cudaMemcpyDefault, g->stream));
+    }
+    GC_CUDA_TRY(cudaEventRecord(e1, g->stream));
+    GC_CUDA_TRY(cudaEventSynchronize(e1));
+    float ms = 0.f;
+    cudaEventElapsedTime(&ms, e0, e1);
+    cudaEventDestroy(e0);
+    cudaEventDestroy(e1);
+    if (!luby && (o->flags & GC_COMPACT) == 0) {
+        // raw colours are < 2RH; they must fit int32 (GC_ERR_TOO_LARGE otherwise)
+        if ((uint64_t)2 * (uint64_t)res.rounds * (uint64_t)H > 0x7FFFFFFFull) {
+            set_error("colours exceed INT32_MAX; use GC_COMPACT");
+            return GC_ERR_TOO_LARGE;
+        }
+    }
+    if (stats) {
+        stats->mode_used = mode;
+        stats->rounds = res.rounds;
+        stats->inner_iterations = res.inner;
+        stats->n_colors = ncol;
+        stats->launches = launches;
+        stats->ms = ms;
+        for (int c = 0; c < 4; ++c) {
+            stats->kernel_ms[c] = prof.ms[c];
+            stats->kernel_launches[c] = prof.launches[c];
+            stats->kernel_bytes[c] = prof.bytes[c];
+        }
+        stats->visits = prof.visits;
+        if (stats->frontier_sizes && stats->frontier_cap > 0 && !luby) {
+            int64_t m = std::min<int64_t>(std::min<int64_t>(stats->frontier_cap, res.rounds),
+                                          g->s.nk_cap);
+            if (m > 0)
+                GC_CUDA_TRY(cudaMemcpy(stats->frontier_sizes, g->s.nk, sizeof(int64_t) * m,
+                                       cudaMemcpyDefault));
+        }
+    }
+    return ncol;
+}
+
+int64_t gc_color(gc_graph *g, uint64_t seed, int32_t variant, int32_t *colors_out) {
+    gc_options o;
+    memset(&o, 0, sizeof(o));
+    o.struct_size = sizeof(o);
+    o.variant = variant;
+    o.seed = seed;
+    return gc_color_ex(g, &o, colors_out, nullptr);
+}
+
+int gc_priorities(uint64_t seed, int32_t j, int64_t v_begin, int64_t count, uint32_t *out) {
+    if (count < 0 || v_begin < 0 || (count > 0 && !out) || j < 0 || j >= GC_MAX_HASHES) {
+        set_error("gc_priorities: bad arguments");
+        return GC_ERR_INVALID_ARG;
+    }
+    int dev = 0, sms = 0;
+    int rc = current_device_ok(&dev, &sms);
+    if (rc) return rc;
+    if (count == 0) return GC_OK;
+    if (is_device_ptr(out)) {
+        rc = launch_priorities(seed, j, v_begin, count, out, 0);
+        if (rc) return rc;
+        GC_CUDA_TRY(cudaStreamSynchronize(0));
+        return GC_OK;
+    }
+    uint32_t *d = nullptr;
+    GC_CUDA_TRY(cudaMalloc(&d, sizeof(uint32_t) * (size_t)count));
+    rc = launch_priorities(seed, j, v_begin, count, d, 0);
+    if (!rc) {
+        cudaError_t e = cudaMemcpy(out, d, sizeof(uint32_t) * (size_t)count, cudaMemcpyDeviceToHost);
+        if (e != cudaSuccess) rc = cuda_fail(e, "gc_priorities copy");
+    }
+    cudaFree(d);
+    return rc;
+}
+
+int64_t gc_count_colors(const int32_t *colors, int64_t n) {
+    if (n < 0 || (n > 0 && !colors)) {
+        set_error("gc_count_colors: bad arguments");
+        return GC_ERR_INVALID_ARG;
+    }
+    if (n == 0) return 0;
+    int dev = 0, sms = 0;
+    int rc = current_device_ok(&dev, &sms);
+    if (rc) return rc;
+    gc_graph tmp;
+    tmp.device = dev;
+    tmp.sm_count = sms;
+    tmp.n = n;
+    const uint32_t *C = reinterpret_cast<const uint32_t *>(colors);
+    uint32_t *dC = nullptr;
+    if (!is_device_ptr(colors)) {
+        GC_CUDA_TRY(cudaMalloc(&dC, sizeof(uint32_t) * (size_t)n));
+        GC_CUDA_TRY(cudaMemcpy(dC, colors, sizeof(uint32_t) * (size_t)n, cudaMemcpyHostToDevice));
+        C = dC;
+    }
+    int64_t launches = 0;
+    int64_t r = GC_OK;
+    cudaError_t e = cudaMalloc(&tmp.s.ctr, kCtrWords * sizeof(unsigned long long));
+    if (e == cudaSuccess) e = cudaMallocHost(&tmp.s.host_pinned, 4096);
+    if (e != cudaSuccess) r = cuda_fail(e, "gc_count_colors alloc");
+    if (r == GC_OK) r = count_colors_device(&tmp, C, n, false, nullptr, &launches);
+    free_scratch(tmp.s);
+    cudaFree(dC);
+    return r;
+}
+
+}  // extern "C"

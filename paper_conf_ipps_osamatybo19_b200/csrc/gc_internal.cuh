@@ -1,0 +1,137 @@
+// gc_internal.cuh -- shared internals of libgc (the CUDA path).  Nothing here
+// is shared with oracle/ (by rule: the oracle is an independent program).
+#pragma once
+
+#include <cuda_runtime.h>
+#include <stdint.h>
+
+#include <string>
+#include <vector>
+
+#include "../../include/gc.h"
+
+#define GC_UNC 0xFFFFFFFFu  // "invalidColor" of Alg.5 L5
+#define GC_MAX_HASHES 16
+
+namespace gc {
+
+// ------------------------------------------------------------------ weights
+// R1: p_j(v) = fmix32(v ^ K_j), K_j = fmix32(fold32(seed) +
+// 0x9E3779B9 * (j + 1)).  fmix32 is MurmurHash3's 32-bit finaliser; it is a
+// bijection on uint32 so weights never tie (R2).
+__host__ __device__ __forceinline__ uint32_t weight_mix(uint32_t x) {
+    x ^= x >> 16;
+    x *= 0x85EBCA6Bu;
+    x ^= x >> 13;
+    x *= 0xC2B2AE35u;
+    x ^= x >> 16;
+    return x;
+}
+
+inline uint32_t weight_key(uint64_t seed, int j) {
+    uint32_t folded = (uint32_t)(seed ^ (seed >> 32));
+    return weight_mix(folded + 0x9E3779B9u * (uint32_t)(j + 1));
+}
+
+struct Keys {
+    uint32_t k[GC_MAX_HASHES];
+};
+
+// ---------------------------------------------------------------- handle
+struct Dist;  // distributed state (gc_dist.cu)
+
+struct Scratch {
+    // all device memory, sized for n (or n_local for the distributed path)
+    uint32_t *C = nullptr;        // colours, GC_UNC = uncoloured
+    uint32_t *F[2] = {nullptr, nullptr};  // frontiers (vertex ids)
+    uint32_t *hub = nullptr;      // per-round hub work list
+    uint32_t *S = nullptr;        // Luby inner-loop state / event stamps
+    uint32_t *W = nullptr;        // event mode: witness pairs (2 per vertex)
+    uint32_t *P = nullptr;        // event mode: resume cursors (2 per vertex)
+    unsigned long long *ctr = nullptr;  // device counters (see gc_sweep.cu)
+    int64_t *nk = nullptr;        // per-round frontier sizes (stats), cap nk_cap
+    int64_t nk_cap = 0;
+    uint32_t *bitmap = nullptr;   // colour-count bitmap
+    int64_t bitmap_words = 0;
+    int64_t *host_pinned = nullptr;  // pinned readback area
+};
+
+}  // namespace gc
+
+struct gc_graph {
+    int device = 0;
+    int64_t n = 0;          // vertices owned (== n_global on one GPU)
+    int64_t n_global = 0;
+    int64_t v_begin = 0;    // owned range start
+    int64_t nnz = 0;
+    int64_t max_deg = 0;
+    int64_t *ro = nullptr;  // device row offsets (local rows)
+    uint32_t *ci = nullptr; // device column indices (global ids)
+    bool owns_csr = true;
+    cudaStream_t stream = 0;
+    gc::Scratch s;
+    gc::Dist *dist = nullptr;
+    int sm_count = 148;
+};
+
+namespace gc {
+
+// ----------------------------------------------------------------- errors
+void set_error(const std::string &msg);
+int cuda_fail(cudaError_t e, const char *what);
+
+#define GC_CUDA_TRY(expr)                                   \
+    do {                                                    \
+        cudaError_t _e = (expr);                            \
+        if (_e != cudaSuccess) return gc::cuda_fail(_e, #expr); \
+    } while (0)
+
+bool is_device_ptr(const void *p);
+
+// ------------------------------------------------------------- launchers
+// GC_PROFILE accumulators (kernel classes: 0 sweep, 1 hub, 2 other)
+struct Profile {
+    bool on = false;
+    double ms[4] = {0, 0, 0, 0};
+    int64_t launches[4] = {0, 0, 0, 0};
+    int64_t bytes[4] = {0, 0, 0, 0};
+    int64_t visits = 0;
+};
+
+// Pool of CUDA events bracketing individual launches in profile mode.
+struct EventTimer {
+    std::vector<cudaEvent_t> ev;
+    std::vector<int> cls;
+    size_t used = 0;
+    ~EventTimer();
+    int begin(cudaStream_t st, int klass);   // records the start event
+    int end(cudaStream_t st);                // records the matching stop event
+    int drain(Profile *p);                   // after a stream sync: add durations
+};
+
+struct RunParams {
+    Profile *prof = nullptr;
+    int H = 1;
+    Keys keys;
+    int32_t thread_deg_max = 8;
+    int32_t hub_deg_min = 4096;
+    int32_t batch_rounds = 0;
+    int64_t max_rounds = 0;
+};
+
+struct RunResult {
+    int64_t rounds = 0;
+    int64_t inner = 0;
+    int64_t launches = 0;
+};
+
+int ensure_scratch(gc_graph *g, bool need_event, bool need_luby);
+int run_sweep_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
+int run_event_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
+int run_luby(gc_graph *g, const RunParams &p, RunResult *r);
+int64_t count_colors_device(gc_graph *g, const uint32_t *C, int64_t n, bool compact,
+                            uint32_t *C_inout, int64_t *launches);
+int launch_priorities(uint64_t seed, int j, int64_t v_begin, int64_t count, uint32_t *out,
+                      cudaStream_t st);
+
+}  // namespace gc

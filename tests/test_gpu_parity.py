@@ -1,0 +1,264 @@
+"""Parity of the CUDA path (libgc through its C ABI) with the CPU oracle.
+
+Bit-exact comparison of colourings (integer work): every test feeds the same
+seeded graph to oracle/ and to libgc and compares element by element.  At the
+bench's full size (R-MAT scale 24) the oracle's O(H*m) local certificate --
+which determines the colouring uniquely (pinned in test_oracle.py) -- checks
+every vertex, alongside the frontier-size trace of a smaller R-MAT.
+"""
+from __future__ import annotations
+
+import random
+
+import numpy as np
+import pytest
+import torch
+
+import graphgen as G
+import oracle as O
+import paper_conf_ipps_osamatybo19_b200 as gcb
+from paper_conf_ipps_osamatybo19_b200 import build as gbuild
+
+pytestmark = pytest.mark.gpu
+
+MODES = [gcb.MODE_SWEEP]  # + MODE_EVENT once implemented
+
+
+@pytest.fixture(scope="module", autouse=True)
+def _built():
+    gbuild.build()
+    gcb.lib()
+
+
+def variant_of(name: str, H: int = 1) -> int:
+    return {"maxmin": gcb.MAXMIN, "luby": gcb.LUBY_MIS}.get(name, gcb.MULTIHASH(H))
+
+
+def oracle_colors(g, seed, variant, H=1):
+    if variant == "luby":
+        return O.color_luby(g, seed)
+    return O.color_maxmin(g, seed, H)
+
+
+def gpu_colors(g, seed, vcode, device_out=False, **kw):
+    with gcb.Graph(g.n, g.row_offsets, g.col_indices) as h:
+        out = torch.empty(g.n, dtype=torch.int32, device="cuda" if device_out else "cpu")
+        out, k, st = h.color(seed, vcode, out, stats=True, **kw)
+        return out.cpu().numpy().view(np.uint32), k, st
+
+
+def supported_modes(vname, H):
+    return [gcb.MODE_SWEEP] if vname == "luby" else MODES
+
+
+# ------------------------------------------------------------- a0 weights
+def test_priorities_bit_exact():
+    for seed in (1, 42, 2**33 + 5):
+        for j in (0, 1, 7, 15):
+            for v0, cnt in ((0, 1000), (2**31 - 500, 1000), (2**32 - 300, 300)):
+                ref = np.array([O.priority(seed, j, (v0 + i) & 0xFFFFFFFF) for i in range(cnt)],
+                               dtype=np.uint32)
+                host = torch.empty(cnt, dtype=torch.int32)
+                gcb.priorities(seed, j, v0, cnt, host)
+                dev = torch.empty(cnt, dtype=torch.int32, device="cuda")
+                gcb.priorities(seed, j, v0, cnt, dev)
+                assert (host.numpy().view(np.uint32) == ref).all()
+                assert (dev.cpu().numpy().view(np.uint32) == ref).all()
+    big = torch.empty(1 << 24, dtype=torch.int32, device="cuda")
+    gcb.priorities(3, 2, 0, 1 << 24, big)
+    assert (big.cpu().numpy().view(np.uint32) == O.priorities(3, 2, 1 << 24)).all()
+
+
+# ------------------------------------------------------ golden and random
+def test_golden_tiny():
+    from test_oracle import load_golden
+    for name, n, edges, variant, expect in load_golden():
+        g = G.csr_from_lists(n, edges)
+        H = int(variant[len("multihash"):]) if variant.startswith("multihash") else 1
+        vname = "multihash" if variant.startswith("multihash") else variant
+        for mode in supported_modes(vname, H):
+            C, k, _ = gpu_colors(g, 1, variant_of(vname, H), mode=mode)
+            assert C.tolist() == expect, (name, mode)
+            assert k == len(set(expect))
+
+
+@pytest.mark.parametrize("vname,H", [("maxmin", 1), ("multihash", 2), ("multihash", 3),
+                                     ("multihash", 16), ("luby", 1)])
+def test_random_small_graphs(vname, H):
+    rng = random.Random(H * 7 + len(vname))
+    for i in range(120):
+        n = rng.randint(0, 300)
+        p = rng.choice([0.0, 0.01, 0.05, 0.2, 0.5])
+        g = G.random_graph(n, p, seed=1000 * H + i)
+        seed = rng.getrandbits(64)
+        ref = oracle_colors(g, seed, vname, H)
+        for mode in supported_modes(vname, H):
+            C, k, st = gpu_colors(g, seed, variant_of(vname, H), mode=mode,
+                                  thread_deg_max=rng.choice([0, 1, 4, 64]),
+                                  hub_deg_min=rng.choice([0, 2, 40, 1 << 20]),
+                                  batch_rounds=rng.choice([0, 1, 3]))
+            assert (C == ref).all(), (i, n, p, mode)
+            assert k == (O.count_colors(ref) if n else 0)
+
+
+# --------------------------------------------------------------- edge cases
+def _csr_tensors(n, pairs):
+    return G.csr_from_pairs(n, torch.tensor([a for a, _ in pairs], dtype=torch.int64),
+                            torch.tensor([b for _, b in pairs], dtype=torch.int64))
+
+
+@pytest.mark.parametrize("mode", MODES)
+def test_adversarial_shapes(mode):
+    cases = [
+        G.csr_from_lists(0, []),
+        G.csr_from_lists(1, []),
+        G.csr_from_lists(33, []),                                 # isolated, n % 32 != 0
+        _csr_tensors(200001, [(0, i) for i in range(1, 200001)]),  # hub star K_{1,200000}
+        G.csr_from_lists(700, [(a, b) for a in range(700) for b in range(a + 1, 700)]),  # clique
+        _csr_tensors(100000, [(i, i + 1) for i in range(99999)]),  # long path
+        G.mesh3d(9, 7, 5),
+    ]
+    for g in cases:
+        for vname, H in (("maxmin", 1), ("multihash", 4), ("luby", 1)):
+            if vname == "luby" and mode != gcb.MODE_SWEEP:
+                continue
+            ref = oracle_colors(g, 11, vname, H)
+            C, k, st = gpu_colors(g, 11, variant_of(vname, H), mode=mode)
+            assert (C == ref).all(), (g.name, vname, H)
+    # the clique needs exactly n/2 rounds
+    g = cases[4]
+    _, k, st = gpu_colors(g, 5, gcb.MAXMIN, mode=mode)
+    assert st.rounds == 350 and k == 700
+
+
+def test_duplicates_and_unsorted_rows():
+    g = G.erdos_renyi(5000, 40000, seed=3)
+    ref = O.color_maxmin(g, 9)
+    # shuffle each row and duplicate some entries: adjacency sets are unchanged
+    ro, ci = g.row_offsets.tolist(), g.col_indices.tolist()
+    rng = random.Random(0)
+    rows = []
+    for v in range(g.n):
+        r = ci[ro[v]:ro[v + 1]]
+        r = r + rng.sample(r, min(len(r), 2))
+        rng.shuffle(r)
+        rows.append(r)
+    nro = [0]
+    for r in rows:
+        nro.append(nro[-1] + len(r))
+    g2 = G.Graph(g.n, torch.tensor(nro, dtype=torch.int64),
+                 torch.tensor([x for r in rows for x in r], dtype=torch.int32))
+    for mode in MODES:
+        C, _, _ = gpu_colors(g2, 9, gcb.MAXMIN, mode=mode)
+        assert (C == ref).all()
+    C, _, _ = gpu_colors(g2, 9, gcb.LUBY_MIS)
+    assert (C == O.color_luby(g, 9)).all()
+
+
+def test_schedule_invariance_and_device_output():
+    g = G.rmat(14, 16, seed=2)
+    ref = O.color_maxmin(g, 1)
+    for mode in MODES:
+        for tdm, hub, b in ((1, 2, 1), (8, 4096, 0), (32, 64, 7), (1 << 20, 1 << 30, 2)):
+            C, _, _ = gpu_colors(g, 1, gcb.MAXMIN, mode=mode, thread_deg_max=tdm,
+                                 hub_deg_min=hub, batch_rounds=b, device_out=True)
+            assert (C == ref).all()
+
+
+def test_errors():
+    ro = torch.tensor([0, 1, 2], dtype=torch.int64)
+    with pytest.raises(gcb.GCError) as e:
+        gcb.Graph(2, ro, torch.tensor([0, 0], dtype=torch.int32))      # self-loop
+    assert e.value.code == -2
+    with pytest.raises(gcb.GCError) as e:
+        gcb.Graph(2, ro, torch.tensor([5, 0], dtype=torch.int32))      # col >= n
+    assert e.value.code == -1
+    with pytest.raises(gcb.GCError) as e:
+        gcb.Graph(3, torch.tensor([0, 1, 1, 1]), torch.tensor([1], dtype=torch.int32),
+                  flags=gcb.VALIDATE)                                   # not symmetric
+    assert e.value.code == -3
+    g = gcb.Graph(2, ro, torch.tensor([1, 0], dtype=torch.int32))
+    with pytest.raises(gcb.GCError):
+        g.color(1, gcb.MULTIHASH(17))
+    with pytest.raises(gcb.GCError):
+        g.color(1, 99)
+    g.close()
+
+
+def test_compact_and_count_colors():
+    g = G.erdos_renyi(20000, 160000, seed=5)
+    raw = O.color_maxmin(g, 2)
+    C, k, _ = gpu_colors(g, 2, gcb.MAXMIN, flags=gcb.COMPACT)
+    assert (C == O.compact_colors(raw)).all()
+    assert k == O.count_colors(raw) == int(C.max()) + 1
+    assert gcb.count_colors(torch.from_numpy(raw.view(np.int32))) == k
+    assert gcb.count_colors(torch.from_numpy(raw.view(np.int32)).cuda()) == k
+
+
+def test_borrow_device_and_stream():
+    g = G.rmat(12, 16, seed=4).to("cuda")
+    ref = O.color_maxmin(g.to("cpu"), 3)
+    s = torch.cuda.Stream()
+    with gcb.Graph(g.n, g.row_offsets, g.col_indices, flags=gcb.BORROW_DEVICE) as h:
+        h.set_stream(s)
+        out = torch.empty(g.n, dtype=torch.int32, device="cuda")
+        with torch.cuda.stream(s):
+            h.color(3, gcb.MAXMIN, out)
+        s.synchronize()
+        assert (out.cpu().numpy().view(np.uint32) == ref).all()
+
+
+# ----------------------------------------------------------- config sizes
+@pytest.mark.parametrize("mode", MODES)
+def test_cfg1_grid(mode):
+    g = G.config_graph("cfg1")
+    ref, R, nk = O.color_maxmin(g, 1, with_stats=True)
+    C, k, st = gpu_colors(g, 1, gcb.MAXMIN, mode=mode, frontier_cap=64)
+    assert (C == ref).all() and st.rounds == R and st.frontier_sizes == nk
+
+
+def test_cfg2_er_luby_and_maxmin():
+    g = G.config_graph("cfg2", device="cuda").to("cpu")
+    ref, ncol, inner = O.color_luby(g, 1, with_stats=True)
+    C, k, st = gpu_colors(g, 1, gcb.LUBY_MIS)
+    assert (C == ref).all() and k == ncol and st.inner_iterations == inner
+    ref2, R, nk = O.color_maxmin(g, 1, with_stats=True)
+    for mode in MODES:
+        C, k, st = gpu_colors(g, 1, gcb.MAXMIN, mode=mode, frontier_cap=4096)
+        assert (C == ref2).all() and st.rounds == R and st.frontier_sizes == nk
+
+
+@pytest.mark.parametrize("H", [1, 2, 4, 8])
+def test_cfg3_mesh_multihash(H):
+    g = G.config_graph("cfg3", device="cuda").to("cpu")
+    ref, R, nk = O.color_maxmin(g, 1, H, with_stats=True)
+    for mode in MODES:
+        C, k, st = gpu_colors(g, 1, gcb.MULTIHASH(H), mode=mode, frontier_cap=4096)
+        assert (C == ref).all() and st.rounds == R and st.frontier_sizes == nk
+
+
+def test_rmat_s18_full_oracle():
+    g = G.rmat(18, 16, seed=1, device="cuda").to("cpu")
+    ref, R, nk = O.color_maxmin(g, 1, with_stats=True)
+    for mode in MODES:
+        C, k, st = gpu_colors(g, 1, gcb.MAXMIN, mode=mode, frontier_cap=8192)
+        assert (C == ref).all() and st.rounds == R and st.frontier_sizes == nk
+    C, k, st = gpu_colors(g, 1, gcb.LUBY_MIS)
+    assert (C == O.color_luby(g, 1)).all()
+    C, k, st = gpu_colors(g, 1, gcb.MULTIHASH(4))
+    assert (C == O.color_maxmin(g, 1, 4)).all()
+
+
+def test_cfg4_rmat_s24_certificate():
+    """Full bench size, bench launch configuration (defaults): the certificate
+    (unique characterisation of the max-min colouring) checks every vertex,
+    plus properness and the 2R identity."""
+    g = G.config_graph("cfg4", device="cuda")
+    with gcb.Graph(g.n, g.row_offsets, g.col_indices, flags=gcb.BORROW_DEVICE) as h:
+        out = torch.empty(g.n, dtype=torch.int32, device="cuda")
+        _, k, st = h.color(1, gcb.MAXMIN, out, stats=True)
+    C = out.cpu().numpy().view(np.uint32)
+    gh = g.to("cpu")
+    assert O.cert_maxmin(gh, 1, 1, C) == 0
+    assert O.check_proper(gh, C) == 0
+    assert k == O.count_colors(C) and k in (2 * st.rounds - 1, 2 * st.rounds)
