@@ -223,6 +223,8 @@ int ensure_scratch(gc_graph *g, bool need_event, bool need_luby) {
     if (need_event && !s.W) {
         GC_CUDA_TRY(cudaMalloc(&s.W, nn * 8));
         GC_CUDA_TRY(cudaMalloc(&s.P, nn * 8));
+        GC_CUDA_TRY(cudaMalloc(&s.Q, nn * 4));
+        GC_CUDA_TRY(cudaMalloc(&s.Q2, nn * 4));
     }
     return GC_OK;
 }
@@ -286,6 +288,8 @@ static void free_scratch(Scratch &s) {
     cudaFree(s.S);
     cudaFree(s.W);
     cudaFree(s.P);
+    cudaFree(s.Q);
+    cudaFree(s.Q2);
     cudaFree(s.ctr);
     cudaFree(s.nk);
     cudaFree(s.bitmap);
@@ -467,7 +471,7 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
 
     const bool luby = kind == GC_LUBY_MIS;
     int mode = o->mode;
-    if (mode == GC_MODE_AUTO) mode = GC_MODE_SWEEP;
+    if (mode == GC_MODE_AUTO) mode = GC_MODE_EVENT;
     if (luby) mode = GC_MODE_SWEEP;
     if (mode == GC_MODE_EVENT && H != 1) mode = GC_MODE_SWEEP;
 

@@ -1,12 +1,554 @@
-// gc_event.cu -- EVENT mode (work-efficient witness/resume sweep); see DESIGN.md.
+// gc_event.cu -- EVENT mode of the max-min colouring (H = 1): the same rounds
+// and the same colours as Alg.5, computed work-efficiently.
+//
+// Why: on power-law graphs the round count reaches thousands (R-MAT s24:
+// 2,518 rounds) while most uncoloured vertices stay blocked for hundreds of
+// rounds.  The paper's ComputeOp re-scans every uncoloured row every round
+// (its "serial for loop" flaw); measured on B200 the
+// sweep mode visits ~335 x nnz entries per colouring at s24.
+//
+// How: v is blocked in round k iff it has an
+// uncoloured neighbour with a larger weight (a "hi witness") and one with a
+// smaller weight (a "lo witness") -- Alg.5 L29-34 leave both colormax and
+// colormin false.  Each blocked vertex keeps one witness per side, W[v], and
+// the row position of each, P[v], chosen as the FIRST qualifying neighbour at
+// or after a cursor.  Weights are fixed and colouring is monotone, so every
+// row entry before the witness is either coloured or on the other side, now
+// and forever; when a witness is coloured the search resumes right after it.
+// v's outcome can only change when one of its witnesses is coloured, so a
+// round evaluates only the vertices whose witness was coloured in the
+// previous round (found by walking the rows of newly coloured vertices).
+// Each side's cursor only moves forward: the whole colouring reads each row
+// O(1) times instead of once per round.
+//
+// Round k: k_eval (vertices of D_k; lane / warp scans) -> k_eval_big (CTA per
+// long remaining scan) -> k_notify (rows of the vertices coloured in round k;
+// lane / warp) -> k_notify_big (rows of long coloured vertices split across
+// the whole grid).  Status test: u is uncoloured at the start of round k iff
+// C[u] >= 2k (as in sweep mode), so in-place colour writes are race-free.
 #include "gc_internal.cuh"
 
 namespace gc {
 
+int fill_u32(uint32_t *p, uint32_t val, int64_t n, cudaStream_t st);
+int ensure_nk(gc_graph *g, int64_t need);
+
+namespace {
+
+constexpr int kBlock = 256;
+constexpr int kBigBlock = 512;
+constexpr unsigned kFull = 0xFFFFFFFFu;
+constexpr uint32_t kNone = 0xFFFFFFFFu;
+
+// counter slots in g->s.ctr used by this mode
+enum : int {
+    kD = 24,      // [24..26] |D_k| rotating k % 3
+    kI = 27,      // [27..29] |I_k| (coloured in round k)
+    kBE = 30,     // [30..32] long-scan queue of round k
+    kBN = 33,     // [33..35] long-row notify queue of round k
+    kRem = 36,    // uncoloured vertices
+    kVisE = 37,   // PROF: entries scanned by k_eval
+    kVisB = 38,   // PROF: entries scanned by k_eval_big
+    kVisN = 39,   // PROF: entries walked by the notify kernels
+    kSumD = 40    // PROF: sum of |D_k|
+};
+
+__device__ __forceinline__ unsigned lane_id() { return threadIdx.x & 31u; }
+
+struct Found {
+    int64_t hpos = -1, lpos = -1;  // absolute edge index of the witness, -1 = none
+    uint32_t hw = kNone, lw = kNone;
+};
+
+// Lane-serial witness search over [min(sh,sl), re).
+__device__ __forceinline__ void lane_search(const uint32_t *__restrict__ ci, const uint32_t *C,
+                                            uint32_t thresh, uint32_t key, uint32_t pv,
+                                            bool need_hi, bool need_lo, int64_t sh, int64_t sl,
+                                            int64_t re, Found &f, uint32_t &nvis) {
+    int64_t s = need_hi ? sh : re;
+    if (need_lo && sl < s) s = sl;
+    for (int64_t e = s; e < re; ++e) {
+        ++nvis;
+        const uint32_t u = ci[e];
+        if (C[u] < thresh) continue;  // coloured before round k
+        const uint32_t pu = weight_mix(u ^ key);
+        if (need_hi && f.hpos < 0 && e >= sh && pu > pv) {
+            f.hpos = e;
+            f.hw = u;
+        }
+        if (need_lo && f.lpos < 0 && e >= sl && pu < pv) {
+            f.lpos = e;
+            f.lw = u;
+        }
+        if ((!need_hi || f.hpos >= 0) && (!need_lo || f.lpos >= 0)) break;
+    }
+}
+
+// Warp-cooperative witness search (all arguments warp-uniform).
+__device__ __forceinline__ void warp_search(const uint32_t *__restrict__ ci, const uint32_t *C,
+                                            uint32_t thresh, uint32_t key, uint32_t pv,
+                                            bool need_hi, bool need_lo, int64_t sh, int64_t sl,
+                                            int64_t re, Found &f, uint32_t &nvis) {
+    const unsigned lane = lane_id();
+    int64_t s = need_hi ? sh : re;
+    if (need_lo && sl < s) s = sl;
+    for (int64_t e0 = s; e0 < re; e0 += 64) {
+        const int64_t e1 = e0 + lane, e2 = e0 + 32 + lane;
+        const uint32_t u1 = e1 < re ? ci[e1] : 0u;
+        const uint32_t u2 = e2 < re ? ci[e2] : 0u;
+        const uint32_t c1 = e1 < re ? C[u1] : 0u;
+        const uint32_t c2 = e2 < re ? C[u2] : 0u;
+        nvis += (e1 < re) + (e2 < re);
+        bool h1 = false, l1 = false, h2 = false, l2 = false;
+        if (e1 < re && c1 >= thresh) {
+            const uint32_t pu = weight_mix(u1 ^ key);
+            h1 = need_hi && e1 >= sh && pu > pv;
+            l1 = need_lo && e1 >= sl && pu < pv;
+        }
+        if (e2 < re && c2 >= thresh) {
+            const uint32_t pu = weight_mix(u2 ^ key);
+            h2 = need_hi && e2 >= sh && pu > pv;
+            l2 = need_lo && e2 >= sl && pu < pv;
+        }
+        if (f.hpos < 0) {
+            unsigned b1 = __ballot_sync(kFull, h1), b2 = __ballot_sync(kFull, h2);
+            if (b1) {
+                int l = __ffs(b1) - 1;
+                f.hpos = e0 + l;
+                f.hw = __shfl_sync(kFull, u1, l);
+            } else if (b2) {
+                int l = __ffs(b2) - 1;
+                f.hpos = e0 + 32 + l;
+                f.hw = __shfl_sync(kFull, u2, l);
+            }
+        }
+        if (f.lpos < 0) {
+            unsigned b1 = __ballot_sync(kFull, l1), b2 = __ballot_sync(kFull, l2);
+            if (b1) {
+                int l = __ffs(b1) - 1;
+                f.lpos = e0 + l;
+                f.lw = __shfl_sync(kFull, u1, l);
+            } else if (b2) {
+                int l = __ffs(b2) - 1;
+                f.lpos = e0 + 32 + l;
+                f.lw = __shfl_sync(kFull, u2, l);
+            }
+        }
+        if ((!need_hi || f.hpos >= 0) && (!need_lo || f.lpos >= 0)) break;
+    }
+}
+
+// Where a vertex of D_k resumes: which sides lost their witness and from where.
+struct Resume {
+    bool need_hi, need_lo;
+    int64_t sh, sl;
+};
+
+__device__ __forceinline__ Resume resume_of(uint32_t v, int64_t rs, bool dense, const uint2 *W,
+                                            const uint2 *P, const uint32_t *C, uint32_t thresh) {
+    Resume r;
+    if (dense) {
+        r.need_hi = r.need_lo = true;
+        r.sh = r.sl = rs;
+    } else {
+        const uint2 w = W[v];
+        const uint2 p = P[v];
+        r.need_hi = C[w.x] < thresh;  // hi witness coloured in an earlier round
+        r.need_lo = C[w.y] < thresh;
+        r.sh = rs + (int64_t)p.x + 1;
+        r.sl = rs + (int64_t)p.y + 1;
+    }
+    return r;
+}
+
+// Commit v after its search: blocked -> store the new witnesses; otherwise
+// colour (Alg.5 L37-42: min wins when both, R9).  Returns true if coloured.
+__device__ __forceinline__ bool settle(uint32_t v, int64_t rs, const Resume &r, const Found &f,
+                                       uint32_t k, uint32_t *C, uint2 *W, uint2 *P) {
+    const bool has_hi = !r.need_hi || f.hpos >= 0;
+    const bool has_lo = !r.need_lo || f.lpos >= 0;
+    if (has_hi && has_lo) {
+        if (r.need_hi && r.need_lo) {
+            W[v] = make_uint2(f.hw, f.lw);
+            P[v] = make_uint2((uint32_t)(f.hpos - rs), (uint32_t)(f.lpos - rs));
+        } else if (r.need_hi) {
+            W[v].x = f.hw;
+            P[v].x = (uint32_t)(f.hpos - rs);
+        } else {
+            W[v].y = f.lw;
+            P[v].y = (uint32_t)(f.lpos - rs);
+        }
+        return false;
+    }
+    C[v] = 2u * k + (has_lo ? 0u : 1u);  // atomic-free: single writer
+    return true;
+}
+
+__device__ __forceinline__ void warp_append(bool pred, uint32_t v, uint32_t *list,
+                                            unsigned long long *counter) {
+    const unsigned m = __ballot_sync(kFull, pred);
+    if (!m) return;
+    const unsigned lane = lane_id();
+    const unsigned leader = __ffs(m) - 1;
+    unsigned long long base = 0;
+    if (lane == leader) base = atomicAdd(counter, (unsigned long long)__popc(m));
+    base = __shfl_sync(kFull, base, leader);
+    if (pred) list[base + __popc(m & ((1u << lane) - 1u))] = v;
+}
+
+template <bool PROF>
+__global__ void __launch_bounds__(kBlock) k_eval(
+    const int64_t *__restrict__ ro, const uint32_t *__restrict__ ci, uint32_t *C, uint2 *W,
+    uint2 *P, const uint32_t *__restrict__ Din, uint32_t *__restrict__ Iout,
+    uint32_t *__restrict__ bigq, unsigned long long *ctr, int64_t *nk, int64_t nk_cap, uint32_t k,
+    uint32_t key, int dense, int64_t n, uint32_t thread_max, uint32_t big_min) {
+    const unsigned long long N = dense ? (unsigned long long)n : ctr[kD + k % 3];
+    if (blockIdx.x == 0 && threadIdx.x == 0) {
+        ctr[kD + (k + 2) % 3] = 0;
+        ctr[kI + (k + 1) % 3] = 0;
+        ctr[kBE + (k + 1) % 3] = 0;
+        ctr[kBN + k % 3] = 0;
+        if ((int64_t)k < nk_cap) nk[k] = (int64_t)ctr[kRem];
+        if (PROF) ctr[kSumD] += N;
+    }
+    const uint32_t thresh = 2u * k;
+    const unsigned lane = lane_id();
+    const unsigned long long stride = (unsigned long long)gridDim.x * blockDim.x;
+    for (unsigned long long base = (unsigned long long)blockIdx.x * blockDim.x + (threadIdx.x & ~31u);
+         base < N; base += stride) {
+        const unsigned long long idx = base + lane;
+        const bool valid = idx < N;
+        uint32_t v = 0;
+        int64_t rs = 0, re = 0;
+        Resume r{false, false, 0, 0};
+        if (valid) {
+            v = dense ? (uint32_t)idx : Din[idx];
+            rs = ro[v];
+            re = ro[v + 1];
+            r = resume_of(v, rs, dense != 0, W, P, C, thresh);
+        }
+        const bool work = valid && (r.need_hi || r.need_lo);
+        int64_t s = r.need_hi ? r.sh : re;
+        if (r.need_lo && r.sl < s) s = r.sl;
+        const int64_t remaining = re - s;
+        const bool small = work && remaining <= (int64_t)thread_max;
+        const bool big = work && !small && remaining >= (int64_t)big_min;
+        const bool mid = work && !small && !big;
+        const uint32_t pv = weight_mix(v ^ key);
+        Found f;
+        uint32_t nvis = 0;
+        if (small) lane_search(ci, C, thresh, key, pv, r.need_hi, r.need_lo, r.sh, r.sl, re, f, nvis);
+        unsigned mm = __ballot_sync(kFull, mid);
+        while (mm) {
+            const int src = __ffs(mm) - 1;
+            mm &= mm - 1;
+            const uint32_t pw = __shfl_sync(kFull, pv, src);
+            const bool nh = __shfl_sync(kFull, r.need_hi, src);
+            const bool nl = __shfl_sync(kFull, r.need_lo, src);
+            const int64_t sh = __shfl_sync(kFull, r.sh, src);
+            const int64_t sl = __shfl_sync(kFull, r.sl, src);
+            const int64_t we = __shfl_sync(kFull, re, src);
+            Found fw;
+            uint32_t wv = 0;
+            warp_search(ci, C, thresh, key, pw, nh, nl, sh, sl, we, fw, wv);
+            if ((int)lane == src) f = fw;
+            if (PROF) nvis += wv;
+        }
+        bool colored = false;
+        if (small || mid) colored = settle(v, rs, r, f, k, C, W, P);
+        warp_append(colored, v, Iout, &ctr[kI + k % 3]);
+        warp_append(big, v, bigq, &ctr[kBE + k % 3]);
+        if (PROF) {
+            const unsigned tot = __reduce_add_sync(kFull, nvis);
+            if (lane == 0 && tot) atomicAdd(&ctr[kVisE], (unsigned long long)tot);
+        }
+    }
+}
+
+// CTA per long remaining scan, early exit per 2048-entry chunk.
+template <bool PROF>
+__global__ void __launch_bounds__(kBigBlock) k_eval_big(
+    const int64_t *__restrict__ ro, const uint32_t *__restrict__ ci, uint32_t *C, uint2 *W,
+    uint2 *P, const uint32_t *__restrict__ bigq, uint32_t *__restrict__ Iout,
+    unsigned long long *ctr, uint32_t k, uint32_t key, int dense) {
+    const unsigned long long nbig = ctr[kBE + k % 3];
+    const uint32_t thresh = 2u * k;
+    __shared__ unsigned long long sh_h, sh_l;  // min absolute position found
+    constexpr int kUnroll = 4;
+    uint32_t nvis = 0;
+    for (unsigned long long i = blockIdx.x; i < nbig; i += gridDim.x) {
+        const uint32_t v = bigq[i];
+        const int64_t rs = ro[v], re = ro[v + 1];
+        const Resume r = resume_of(v, rs, dense != 0, W, P, C, thresh);
+        const uint32_t pv = weight_mix(v ^ key);
+        if (threadIdx.x == 0) {
+            sh_h = ~0ull;
+            sh_l = ~0ull;
+        }
+        __syncthreads();
+        int64_t s = r.need_hi ? r.sh : re;
+        if (r.need_lo && r.sl < s) s = r.sl;
+        unsigned long long H = ~0ull, L = ~0ull;
+        for (int64_t e0 = s; e0 < re; e0 += (int64_t)blockDim.x * kUnroll) {
+            uint32_t u[kUnroll], c[kUnroll];
+#pragma unroll
+            for (int q = 0; q < kUnroll; ++q) {
+                const int64_t e = e0 + threadIdx.x + (int64_t)q * blockDim.x;
+                u[q] = e < re ? ci[e] : 0u;
+            }
+#pragma unroll
+            for (int q = 0; q < kUnroll; ++q) {
+                const int64_t e = e0 + threadIdx.x + (int64_t)q * blockDim.x;
+                c[q] = e < re ? C[u[q]] : 0u;
+            }
+            uint32_t rh = 0xFFFFFFFFu, rl = 0xFFFFFFFFu;  // first hit, relative to e0
+#pragma unroll
+            for (int q = 0; q < kUnroll; ++q) {
+                const int64_t e = e0 + threadIdx.x + (int64_t)q * blockDim.x;
+                if (PROF) nvis += e < re;
+                if (e < re && c[q] >= thresh) {
+                    const uint32_t pu = weight_mix(u[q] ^ key);
+                    const uint32_t rel = (uint32_t)(e - e0);
+                    if (r.need_hi && e >= r.sh && pu > pv) rh = min(rh, rel);
+                    if (r.need_lo && e >= r.sl && pu < pv) rl = min(rl, rel);
+                }
+            }
+            rh = __reduce_min_sync(kFull, rh);
+            rl = __reduce_min_sync(kFull, rl);
+            const unsigned long long mh = rh == 0xFFFFFFFFu ? ~0ull : (unsigned long long)(e0 + rh);
+            const unsigned long long ml = rl == 0xFFFFFFFFu ? ~0ull : (unsigned long long)(e0 + rl);
+            if ((threadIdx.x & 31) == 0) {
+                if (mh != ~0ull) atomicMin(&sh_h, mh);
+                if (ml != ~0ull) atomicMin(&sh_l, ml);
+            }
+            __syncthreads();
+            H = sh_h;
+            L = sh_l;
+            __syncthreads();
+            if ((!r.need_hi || H != ~0ull) && (!r.need_lo || L != ~0ull)) break;
+        }
+        if (threadIdx.x == 0) {
+            Found f;
+            if (H != ~0ull) {
+                f.hpos = (int64_t)H;
+                f.hw = ci[H];
+            }
+            if (L != ~0ull) {
+                f.lpos = (int64_t)L;
+                f.lw = ci[L];
+            }
+            if (settle(v, rs, r, f, k, C, W, P)) {
+                const unsigned long long pos = atomicAdd(&ctr[kI + k % 3], 1ull);
+                Iout[pos] = v;
+            }
+        }
+        __syncthreads();
+    }
+    if (PROF) {
+        const unsigned tot = __reduce_add_sync(kFull, nvis);
+        if ((threadIdx.x & 31) == 0 && tot) atomicAdd(&ctr[kVisB], (unsigned long long)tot);
+    }
+}
+
+// Neighbour w of a vertex u coloured in round k must be re-evaluated in
+// round k+1 iff it is uncoloured and u was one of its witnesses.  The stamp
+// S[w] (round+1 of its last enqueue) removes duplicates (duplicate CSR entries,
+// or both witnesses coloured in the same round).
+__device__ __forceinline__ bool wake(uint32_t w, uint32_t u, uint32_t k, const uint32_t *C,
+                                     const uint2 *W, uint32_t *S) {
+    if (C[w] != GC_UNC) return false;
+    const uint2 ww = W[w];
+    if (ww.x != u && ww.y != u) return false;
+    return atomicMax(&S[w], k + 1u) < k + 1u;
+}
+
+template <bool PROF>
+__global__ void __launch_bounds__(kBlock) k_notify(
+    const int64_t *__restrict__ ro, const uint32_t *__restrict__ ci, const uint32_t *C,
+    const uint2 *W, uint32_t *S, const uint32_t *__restrict__ Iin, uint32_t *__restrict__ Dout,
+    uint32_t *__restrict__ bigq, unsigned long long *ctr, uint32_t k, uint32_t thread_max,
+    uint32_t big_min) {
+    const unsigned long long cnt = ctr[kI + k % 3];
+    if (blockIdx.x == 0 && threadIdx.x == 0) ctr[kRem] -= cnt;
+    unsigned long long *dcount = &ctr[kD + (k + 1) % 3];
+    const unsigned lane = lane_id();
+    uint32_t nvis = 0;
+    const unsigned long long stride = (unsigned long long)gridDim.x * blockDim.x;
+    for (unsigned long long base = (unsigned long long)blockIdx.x * blockDim.x + (threadIdx.x & ~31u);
+         base < cnt; base += stride) {
+        const unsigned long long idx = base + lane;
+        const bool valid = idx < cnt;
+        uint32_t u = 0;
+        int64_t rs = 0, re = 0;
+        if (valid) {
+            u = Iin[idx];
+            rs = ro[u];
+            re = ro[u + 1];
+        }
+        const int64_t deg = re - rs;
+        const bool small = valid && deg <= (int64_t)thread_max;
+        const bool big = valid && !small && deg >= (int64_t)big_min;
+        const bool mid = valid && !small && !big;
+        if (small) {
+            for (int64_t e = rs; e < re; ++e) {
+                const uint32_t w = ci[e];
+                if (wake(w, u, k, C, W, S)) Dout[atomicAdd(dcount, 1ull)] = w;
+            }
+            if (PROF) nvis += (uint32_t)deg;
+        }
+        unsigned mm = __ballot_sync(kFull, mid);
+        while (mm) {
+            const int src = __ffs(mm) - 1;
+            mm &= mm - 1;
+            const uint32_t uu = __shfl_sync(kFull, u, src);
+            const int64_t ws = __shfl_sync(kFull, rs, src);
+            const int64_t we = __shfl_sync(kFull, re, src);
+            for (int64_t e0 = ws; e0 < we; e0 += 32) {
+                const int64_t e = e0 + lane;
+                bool wk = false;
+                uint32_t w = 0;
+                if (e < we) {
+                    w = ci[e];
+                    wk = wake(w, uu, k, C, W, S);
+                }
+                warp_append(wk, w, Dout, dcount);
+            }
+            if (PROF && lane == 0) nvis += (uint32_t)(we - ws);
+        }
+        warp_append(big, u, bigq, &ctr[kBN + k % 3]);
+    }
+    if (PROF) {
+        const unsigned tot = __reduce_add_sync(kFull, nvis);
+        if (lane == 0 && tot) atomicAdd(&ctr[kVisN], (unsigned long long)tot);
+    }
+}
+
+// Rows of long coloured vertices, split across the whole grid.
+template <bool PROF>
+__global__ void __launch_bounds__(kBlock) k_notify_big(
+    const int64_t *__restrict__ ro, const uint32_t *__restrict__ ci, const uint32_t *C,
+    const uint2 *W, uint32_t *S, const uint32_t *__restrict__ bigq, uint32_t *__restrict__ Dout,
+    unsigned long long *ctr, uint32_t k) {
+    const unsigned long long nbig = ctr[kBN + k % 3];
+    unsigned long long *dcount = &ctr[kD + (k + 1) % 3];
+    uint32_t nvis = 0;
+    for (unsigned long long i = 0; i < nbig; ++i) {
+        const uint32_t u = bigq[i];
+        const int64_t rs = ro[u], re = ro[u + 1];
+        for (int64_t e = rs + (int64_t)blockIdx.x * blockDim.x + threadIdx.x; e < re;
+             e += (int64_t)gridDim.x * blockDim.x) {
+            const uint32_t w = ci[e];
+            if (PROF) ++nvis;
+            if (wake(w, u, k, C, W, S)) Dout[atomicAdd(dcount, 1ull)] = w;
+        }
+    }
+    if (PROF) {
+        const unsigned tot = __reduce_add_sync(kFull, nvis);
+        if ((threadIdx.x & 31) == 0 && tot) atomicAdd(&ctr[kVisN], (unsigned long long)tot);
+    }
+}
+
+template <bool PROF>
+int launch_round(gc_graph *g, const RunParams &p, uint32_t k, int grid, int grid_dense,
+                 EventTimer *tm) {
+    Scratch &s = g->s;
+    uint2 *W = reinterpret_cast<uint2 *>(s.W);
+    uint2 *P = reinterpret_cast<uint2 *>(s.P);
+    const uint32_t key = p.keys.k[0];
+    const int dense = k == 0 ? 1 : 0;
+    uint32_t *D[2] = {s.F[0], s.F[1]};
+    uint32_t *I = s.hub;
+    int rc;
+    if (PROF && (rc = tm->begin(g->stream, 0))) return rc;
+    k_eval<PROF><<<dense ? grid_dense : grid, kBlock, 0, g->stream>>>(
+        g->ro, g->ci, s.C, W, P, D[k % 2], I, s.Q, s.ctr, s.nk, s.nk_cap, k, key, dense, g->n,
+        (uint32_t)p.thread_deg_max, (uint32_t)p.hub_deg_min);
+    if (PROF && (rc = tm->end(g->stream))) return rc;
+    if (PROF && (rc = tm->begin(g->stream, 1))) return rc;
+    k_eval_big<PROF><<<g->sm_count * 2, kBigBlock, 0, g->stream>>>(g->ro, g->ci, s.C, W, P, s.Q, I,
+                                                                   s.ctr, k, key, dense);
+    if (PROF && (rc = tm->end(g->stream))) return rc;
+    if (PROF && (rc = tm->begin(g->stream, 2))) return rc;
+    k_notify<PROF><<<grid, kBlock, 0, g->stream>>>(g->ro, g->ci, s.C, W, s.S, I, D[(k + 1) % 2],
+                                                   s.Q2, s.ctr, k, (uint32_t)p.thread_deg_max,
+                                                   (uint32_t)p.hub_deg_min);
+    k_notify_big<PROF><<<g->sm_count * 4, kBlock, 0, g->stream>>>(g->ro, g->ci, s.C, W, s.S, s.Q2,
+                                                                  D[(k + 1) % 2], s.ctr, k);
+    if (PROF && (rc = tm->end(g->stream))) return rc;
+    return GC_OK;
+}
+
+}  // namespace
+
 int run_event_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
-    (void)g; (void)p; (void)r;
-    set_error("GC_MODE_EVENT is not implemented yet");
-    return GC_ERR_INVALID_ARG;
+    Scratch &s = g->s;
+    const int64_t n = g->n;
+    r->rounds = r->inner = r->launches = 0;
+    if (n == 0) return GC_OK;
+    int rc = fill_u32(s.C, GC_UNC, n, g->stream);  // Alg.5 L5
+    if (rc) return rc;
+    GC_CUDA_TRY(cudaMemsetAsync(s.S, 0, sizeof(uint32_t) * (size_t)n, g->stream));
+    GC_CUDA_TRY(cudaMemsetAsync(s.ctr, 0, 48 * sizeof(unsigned long long), g->stream));
+    const unsigned long long rem = (unsigned long long)n;
+    GC_CUDA_TRY(cudaMemcpyAsync(s.ctr + kRem, &rem, sizeof(rem), cudaMemcpyHostToDevice, g->stream));
+    r->launches += 1;
+    const int grid = g->sm_count * 4;
+    const int grid_dense =
+        (int)std::max<int64_t>(1, std::min<int64_t>((n + kBlock - 1) / kBlock, (int64_t)g->sm_count * 8));
+    const bool prof = p.prof && p.prof->on;
+    EventTimer tm;
+    int64_t k = 0;
+    int64_t batch = p.batch_rounds > 0 ? p.batch_rounds : 8;
+    for (;;) {
+        rc = ensure_nk(g, k + batch + 1);
+        if (rc) return rc;
+        for (int64_t b = 0; b < batch; ++b, ++k) {
+            rc = prof ? launch_round<true>(g, p, (uint32_t)k, grid, grid_dense, &tm)
+                      : launch_round<false>(g, p, (uint32_t)k, grid, grid_dense, &tm);
+            if (rc) return rc;
+            r->launches += 4;
+        }
+        GC_CUDA_TRY(cudaGetLastError());
+        GC_CUDA_TRY(cudaMemcpyAsync(s.host_pinned, s.nk + (k - batch), sizeof(int64_t) * batch,
+                                    cudaMemcpyDeviceToHost, g->stream));
+        GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
+        if (prof && (rc = tm.drain(p.prof))) return rc;
+        int64_t done_at = -1;
+        for (int64_t b = 0; b < batch; ++b)
+            if (s.host_pinned[b] == 0) {
+                done_at = k - batch + b;
+                break;
+            }
+        if (done_at >= 0) {
+            r->rounds = done_at;
+            break;
+        }
+        if (p.max_rounds > 0 && k >= p.max_rounds) {
+            set_error("max-min colouring exceeded the round limit");
+            return GC_ERR_TOO_LARGE;
+        }
+        if (p.batch_rounds <= 0) batch = std::min<int64_t>(batch * 2, 512);
+    }
+    r->inner = r->rounds;
+    if (prof) {
+        unsigned long long c[8];
+        GC_CUDA_TRY(cudaMemcpy(c, s.ctr + kVisE, sizeof(c), cudaMemcpyDeviceToHost));
+        const int64_t visE = (int64_t)c[0], visB = (int64_t)c[1], visN = (int64_t)c[2];
+        const int64_t sumD = (int64_t)c[3];
+        // algorithmic bytes: eval reads D (4 B), the
+        // row offsets (16 B) and the witness state (16 B; not in the dense
+        // round 0) per evaluated vertex, 4 B per scanned entry, and writes
+        // either the witness state (16 B) or the colour + I entry (8 B);
+        // notify reads I (4 B) and the row offsets (16 B) per coloured vertex
+        // and 4 B per walked entry.
+        const int64_t evalB = 4 * (sumD - n) + 16 * sumD + 16 * (sumD - n) + 4 * visE +
+                              16 * (sumD - n) + 8 * n;
+        p.prof->bytes[0] += evalB;
+        p.prof->bytes[1] += 4 * visB;
+        p.prof->bytes[2] += 20 * n + 4 * visN;
+        p.prof->visits += visE + visB;
+    }
+    return GC_OK;
 }
 
 }  // namespace gc

@@ -44,7 +44,9 @@ struct Scratch {
     // all device memory, sized for n (or n_local for the distributed path)
     uint32_t *C = nullptr;        // colours, GC_UNC = uncoloured
     uint32_t *F[2] = {nullptr, nullptr};  // frontiers (vertex ids)
-    uint32_t *hub = nullptr;      // per-round hub work list
+    uint32_t *hub = nullptr;      // per-round hub work list / event: coloured list I_k
+    uint32_t *Q = nullptr;        // event mode: long-scan queue
+    uint32_t *Q2 = nullptr;       // event mode: long-row notify queue
     uint32_t *S = nullptr;        // Luby inner-loop state / event stamps
     uint32_t *W = nullptr;        // event mode: witness pairs (2 per vertex)
     uint32_t *P = nullptr;        // event mode: resume cursors (2 per vertex)

@@ -122,7 +122,7 @@ __global__ void __launch_bounds__(kBlock) k_sweep(
         }
         const int64_t deg = re - rs;
         const bool small = valid && deg <= (int64_t)thread_max;
-        const bool big = valid && deg >= (int64_t)hub_min;
+        const bool big = valid && !small && deg >= (int64_t)hub_min;
         const bool mid = valid && !small && !big;
         uint32_t pv[HT > 0 ? HT : GC_MAX_HASHES];
         own_weights<HT>(v, keys, nh, pv);
