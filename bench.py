@@ -277,7 +277,10 @@ def main():
         torch.cuda.synchronize()
         peak, peak_src = measured_peaks()
         cls = max(range(4), key=lambda c: sp.kernel_ms[c])
-        name = {0: "sweep", 1: "hub", 2: "other", 3: "other"}[cls]
+        names = ({0: "k_eval", 1: "k_eval_big", 2: "k_notify", 3: "k_notify_big"}
+                 if sp.mode_used == gcb.MODE_EVENT else
+                 {0: "k_sweep", 1: "k_hub", 2: "other", 3: "other"})
+        name = names[cls]
         kms, kl, kb = sp.kernel_ms[cls], sp.kernel_launches[cls], sp.kernel_bytes[cls]
         achieved = (kb / 1e9) / (kms / 1e3) if kms > 0 else 0.0
         roof = {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
@@ -285,7 +288,10 @@ def main():
                 "kernel": name, "launches": kl, "avg_launch_us": 1e3 * kms / max(kl, 1),
                 "bytes_per_launch": kb / max(kl, 1), "kernel_share_of_step":
                 kms / max(sp.ms, 1e-9), "peak_source": peak_src,
-                "visits": sp.visits, "profiled_ms": sp.ms}
+                "visits": sp.visits, "profiled_ms": sp.ms,
+                "classes": {names[c]: {"ms": sp.kernel_ms[c], "launches": sp.kernel_launches[c],
+                                       "bytes": sp.kernel_bytes[c]} for c in range(4)
+                            if sp.kernel_launches[c]}}
 
     # ---- end to end through the C ABI with host buffers
     e2e = None

@@ -224,7 +224,8 @@ int ensure_scratch(gc_graph *g, bool need_event, bool need_luby) {
         GC_CUDA_TRY(cudaMalloc(&s.W, nn * 8));
         GC_CUDA_TRY(cudaMalloc(&s.P, nn * 8));
         GC_CUDA_TRY(cudaMalloc(&s.Q, nn * 4));
-        GC_CUDA_TRY(cudaMalloc(&s.Q2, nn * 4));
+        // long-row notify items (u, segment): at most n + nnz/256 per round
+        GC_CUDA_TRY(cudaMalloc(&s.Q2, (nn + (size_t)g->nnz / 256 + 1) * 8));
     }
     return GC_OK;
 }

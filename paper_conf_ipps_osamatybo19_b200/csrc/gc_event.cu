@@ -39,6 +39,7 @@ constexpr int kBlock = 256;
 constexpr int kBigBlock = 512;
 constexpr unsigned kFull = 0xFFFFFFFFu;
 constexpr uint32_t kNone = 0xFFFFFFFFu;
+constexpr int kSeg = 256;  // entries per long-row notify item (8 per lane)
 
 // counter slots in g->s.ctr used by this mode
 enum : int {
@@ -366,7 +367,7 @@ template <bool PROF>
 __global__ void __launch_bounds__(kBlock) k_notify(
     const int64_t *__restrict__ ro, const uint32_t *__restrict__ ci, const uint32_t *C,
     const uint2 *W, uint32_t *S, const uint32_t *__restrict__ Iin, uint32_t *__restrict__ Dout,
-    uint32_t *__restrict__ bigq, unsigned long long *ctr, uint32_t k, uint32_t thread_max,
+    uint2 *__restrict__ bigq, unsigned long long *ctr, uint32_t k, uint32_t thread_max,
     uint32_t big_min) {
     const unsigned long long cnt = ctr[kI + k % 3];
     if (blockIdx.x == 0 && threadIdx.x == 0) ctr[kRem] -= cnt;
@@ -415,7 +416,19 @@ __global__ void __launch_bounds__(kBlock) k_notify(
             }
             if (PROF && lane == 0) nvis += (uint32_t)(we - ws);
         }
-        warp_append(big, u, bigq, &ctr[kBN + k % 3]);
+        // long rows: one work item per kSeg-entry segment, spread over the grid
+        unsigned bm = __ballot_sync(kFull, big);
+        while (bm) {
+            const int src = __ffs(bm) - 1;
+            bm &= bm - 1;
+            const uint32_t uu = __shfl_sync(kFull, u, src);
+            const int64_t dg = __shfl_sync(kFull, deg, src);
+            const uint32_t nseg = (uint32_t)((dg + kSeg - 1) / kSeg);
+            unsigned long long b0 = 0;
+            if (lane == 0) b0 = atomicAdd(&ctr[kBN + k % 3], (unsigned long long)nseg);
+            b0 = __shfl_sync(kFull, b0, 0);
+            for (uint32_t q = lane; q < nseg; q += 32) bigq[b0 + q] = make_uint2(uu, q);
+        }
     }
     if (PROF) {
         const unsigned tot = __reduce_add_sync(kFull, nvis);
@@ -423,28 +436,39 @@ __global__ void __launch_bounds__(kBlock) k_notify(
     }
 }
 
-// Rows of long coloured vertices, split across the whole grid.
+// Segments of long coloured rows: one warp per kSeg-entry segment.
 template <bool PROF>
 __global__ void __launch_bounds__(kBlock) k_notify_big(
     const int64_t *__restrict__ ro, const uint32_t *__restrict__ ci, const uint32_t *C,
-    const uint2 *W, uint32_t *S, const uint32_t *__restrict__ bigq, uint32_t *__restrict__ Dout,
+    const uint2 *W, uint32_t *S, const uint2 *__restrict__ bigq, uint32_t *__restrict__ Dout,
     unsigned long long *ctr, uint32_t k) {
-    const unsigned long long nbig = ctr[kBN + k % 3];
+    const unsigned long long nitems = ctr[kBN + k % 3];
     unsigned long long *dcount = &ctr[kD + (k + 1) % 3];
+    const unsigned lane = lane_id();
     uint32_t nvis = 0;
-    for (unsigned long long i = 0; i < nbig; ++i) {
-        const uint32_t u = bigq[i];
-        const int64_t rs = ro[u], re = ro[u + 1];
-        for (int64_t e = rs + (int64_t)blockIdx.x * blockDim.x + threadIdx.x; e < re;
-             e += (int64_t)gridDim.x * blockDim.x) {
-            const uint32_t w = ci[e];
-            if (PROF) ++nvis;
-            if (wake(w, u, k, C, W, S)) Dout[atomicAdd(dcount, 1ull)] = w;
+    const unsigned long long warp0 = ((unsigned long long)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+    const unsigned long long nwarps = ((unsigned long long)gridDim.x * blockDim.x) >> 5;
+    for (unsigned long long it = warp0; it < nitems; it += nwarps) {
+        const uint2 item = bigq[it];
+        const uint32_t u = item.x;
+        const int64_t rs = ro[u] + (int64_t)item.y * kSeg;
+        const int64_t re = min(ro[u + 1], rs + (int64_t)kSeg);
+        uint32_t w[kSeg / 32];
+#pragma unroll
+        for (int q = 0; q < kSeg / 32; ++q) {
+            const int64_t e = rs + q * 32 + lane;
+            w[q] = e < re ? ci[e] : 0xFFFFFFFFu;
         }
+#pragma unroll
+        for (int q = 0; q < kSeg / 32; ++q) {
+            const bool wk = w[q] != 0xFFFFFFFFu && wake(w[q], u, k, C, W, S);
+            warp_append(wk, w[q], Dout, dcount);
+        }
+        if (PROF && lane == 0) nvis += (uint32_t)(re - rs);
     }
     if (PROF) {
         const unsigned tot = __reduce_add_sync(kFull, nvis);
-        if ((threadIdx.x & 31) == 0 && tot) atomicAdd(&ctr[kVisN], (unsigned long long)tot);
+        if (lane == 0 && tot) atomicAdd(&ctr[kVisN], (unsigned long long)tot);
     }
 }
 
@@ -469,10 +493,13 @@ int launch_round(gc_graph *g, const RunParams &p, uint32_t k, int grid, int grid
                                                                    s.ctr, k, key, dense);
     if (PROF && (rc = tm->end(g->stream))) return rc;
     if (PROF && (rc = tm->begin(g->stream, 2))) return rc;
+    uint2 *Q2 = reinterpret_cast<uint2 *>(s.Q2);
     k_notify<PROF><<<grid, kBlock, 0, g->stream>>>(g->ro, g->ci, s.C, W, s.S, I, D[(k + 1) % 2],
-                                                   s.Q2, s.ctr, k, (uint32_t)p.thread_deg_max,
-                                                   (uint32_t)p.hub_deg_min);
-    k_notify_big<PROF><<<g->sm_count * 4, kBlock, 0, g->stream>>>(g->ro, g->ci, s.C, W, s.S, s.Q2,
+                                                   Q2, s.ctr, k, (uint32_t)p.thread_deg_max,
+                                                   (uint32_t)std::min(p.hub_deg_min, 4 * kSeg));
+    if (PROF && (rc = tm->end(g->stream))) return rc;
+    if (PROF && (rc = tm->begin(g->stream, 3))) return rc;
+    k_notify_big<PROF><<<g->sm_count * 8, kBlock, 0, g->stream>>>(g->ro, g->ci, s.C, W, s.S, Q2,
                                                                   D[(k + 1) % 2], s.ctr, k);
     if (PROF && (rc = tm->end(g->stream))) return rc;
     return GC_OK;
@@ -545,7 +572,7 @@ int run_event_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
                               16 * (sumD - n) + 8 * n;
         p.prof->bytes[0] += evalB;
         p.prof->bytes[1] += 4 * visB;
-        p.prof->bytes[2] += 20 * n + 4 * visN;
+        p.prof->bytes[2] += 20 * n + 4 * visN;  // notify + notify_big (walked entries)
         p.prof->visits += visE + visB;
     }
     return GC_OK;

@@ -222,8 +222,9 @@ __global__ void __launch_bounds__(512) k_hub(const int64_t *__restrict__ ro,
             }
 #pragma unroll
             for (int q = 0; q < kUnroll; ++q) {
-                if (PROF) nvis += (e0 + threadIdx.x + (int64_t)q * blockDim.x) < re;
-                if (c[q] >= thresh) visit<HT>(u[q], pv, keys, nh, h, l);
+                const bool in_row = (e0 + threadIdx.x + (int64_t)q * blockDim.x) < re;
+                if (PROF) nvis += in_row;
+                if (in_row && c[q] >= thresh) visit<HT>(u[q], pv, keys, nh, h, l);
             }
             h = __reduce_or_sync(kFull, h);
             l = __reduce_or_sync(kFull, l);
