@@ -224,8 +224,8 @@ int ensure_scratch(gc_graph *g, bool need_event, bool need_luby) {
         GC_CUDA_TRY(cudaMalloc(&s.W, nn * 8));
         GC_CUDA_TRY(cudaMalloc(&s.P, nn * 8));
         GC_CUDA_TRY(cudaMalloc(&s.Q, nn * 4));
-        // long-row notify items (u, segment): at most n + nnz/256 per round
-        GC_CUDA_TRY(cudaMalloc(&s.Q2, (nn + (size_t)g->nnz / 256 + 1) * 8));
+        // long-row notify items (u, segment): at most n + nnz/128 per round
+        GC_CUDA_TRY(cudaMalloc(&s.Q2, (nn + (size_t)g->nnz / 128 + 1) * 8));
     }
     return GC_OK;
 }
@@ -483,6 +483,7 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     for (int j = 0; j < H; ++j) p.keys.k[j] = weight_key(o->seed, j);
     p.thread_deg_max = o->thread_deg_max > 0 ? o->thread_deg_max : 8;
     p.hub_deg_min = o->hub_deg_min > 0 ? o->hub_deg_min : 4096;
+    p.eval_big_min = o->hub_deg_min > 0 ? o->hub_deg_min : 256;
     p.batch_rounds = o->batch_rounds;
     p.max_rounds = (int64_t)(0x7FFFFFFFll / (2 * H)) + 1;
     Profile prof;

@@ -39,7 +39,7 @@ constexpr int kBlock = 256;
 constexpr int kBigBlock = 512;
 constexpr unsigned kFull = 0xFFFFFFFFu;
 constexpr uint32_t kNone = 0xFFFFFFFFu;
-constexpr int kSeg = 256;  // entries per long-row notify item (8 per lane)
+constexpr int kSeg = 128;  // entries per long-row notify item (4 per lane)
 
 // counter slots in g->s.ctr used by this mode
 enum : int {
@@ -214,6 +214,35 @@ __global__ void __launch_bounds__(kBlock) k_eval(
     }
     const uint32_t thresh = 2u * k;
     const unsigned lane = lane_id();
+    const unsigned long long nwarps = ((unsigned long long)gridDim.x * blockDim.x) >> 5;
+    const unsigned long long warp0 = ((unsigned long long)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+    if (!dense && N <= nwarps) {
+        // few vertices (the common late round): one warp per vertex, so the
+        // scans of different vertices run in parallel instead of in one warp
+        if (warp0 < N) {
+            const uint32_t v = Din[warp0];
+            const int64_t rs = ro[v], re = ro[v + 1];
+            const Resume r = resume_of(v, rs, false, W, P, C, thresh);
+            int64_t s = r.need_hi ? r.sh : re;
+            if (r.need_lo && r.sl < s) s = r.sl;
+            const bool work = r.need_hi || r.need_lo;
+            const bool big = work && re - s >= (int64_t)big_min;
+            uint32_t nvis = 0;
+            if (work && !big) {
+                Found f;
+                warp_search(ci, C, thresh, key, weight_mix(v ^ key), r.need_hi, r.need_lo, r.sh,
+                            r.sl, re, f, nvis);
+                if (lane == 0 && settle(v, rs, r, f, k, C, W, P))
+                    Iout[atomicAdd(&ctr[kI + k % 3], 1ull)] = v;
+            }
+            if (big && lane == 0) bigq[atomicAdd(&ctr[kBE + k % 3], 1ull)] = v;
+            if (PROF) {
+                const unsigned tot = __reduce_add_sync(kFull, nvis);
+                if (lane == 0 && tot) atomicAdd(&ctr[kVisE], (unsigned long long)tot);
+            }
+        }
+        return;
+    }
     const unsigned long long stride = (unsigned long long)gridDim.x * blockDim.x;
     for (unsigned long long base = (unsigned long long)blockIdx.x * blockDim.x + (threadIdx.x & ~31u);
          base < N; base += stride) {
@@ -388,33 +417,13 @@ __global__ void __launch_bounds__(kBlock) k_notify(
         }
         const int64_t deg = re - rs;
         const bool small = valid && deg <= (int64_t)thread_max;
-        const bool big = valid && !small && deg >= (int64_t)big_min;
-        const bool mid = valid && !small && !big;
+        const bool big = valid && !small;
         if (small) {
             for (int64_t e = rs; e < re; ++e) {
                 const uint32_t w = ci[e];
                 if (wake(w, u, k, C, W, S)) Dout[atomicAdd(dcount, 1ull)] = w;
             }
             if (PROF) nvis += (uint32_t)deg;
-        }
-        unsigned mm = __ballot_sync(kFull, mid);
-        while (mm) {
-            const int src = __ffs(mm) - 1;
-            mm &= mm - 1;
-            const uint32_t uu = __shfl_sync(kFull, u, src);
-            const int64_t ws = __shfl_sync(kFull, rs, src);
-            const int64_t we = __shfl_sync(kFull, re, src);
-            for (int64_t e0 = ws; e0 < we; e0 += 32) {
-                const int64_t e = e0 + lane;
-                bool wk = false;
-                uint32_t w = 0;
-                if (e < we) {
-                    w = ci[e];
-                    wk = wake(w, uu, k, C, W, S);
-                }
-                warp_append(wk, w, Dout, dcount);
-            }
-            if (PROF && lane == 0) nvis += (uint32_t)(we - ws);
         }
         // long rows: one work item per kSeg-entry segment, spread over the grid
         unsigned bm = __ballot_sync(kFull, big);
@@ -486,7 +495,7 @@ int launch_round(gc_graph *g, const RunParams &p, uint32_t k, int grid, int grid
     if (PROF && (rc = tm->begin(g->stream, 0))) return rc;
     k_eval<PROF><<<dense ? grid_dense : grid, kBlock, 0, g->stream>>>(
         g->ro, g->ci, s.C, W, P, D[k % 2], I, s.Q, s.ctr, s.nk, s.nk_cap, k, key, dense, g->n,
-        (uint32_t)p.thread_deg_max, (uint32_t)p.hub_deg_min);
+        (uint32_t)p.thread_deg_max, (uint32_t)p.eval_big_min);
     if (PROF && (rc = tm->end(g->stream))) return rc;
     if (PROF && (rc = tm->begin(g->stream, 1))) return rc;
     k_eval_big<PROF><<<g->sm_count * 2, kBigBlock, 0, g->stream>>>(g->ro, g->ci, s.C, W, P, s.Q, I,
@@ -495,8 +504,7 @@ int launch_round(gc_graph *g, const RunParams &p, uint32_t k, int grid, int grid
     if (PROF && (rc = tm->begin(g->stream, 2))) return rc;
     uint2 *Q2 = reinterpret_cast<uint2 *>(s.Q2);
     k_notify<PROF><<<grid, kBlock, 0, g->stream>>>(g->ro, g->ci, s.C, W, s.S, I, D[(k + 1) % 2],
-                                                   Q2, s.ctr, k, (uint32_t)p.thread_deg_max,
-                                                   (uint32_t)std::min(p.hub_deg_min, 4 * kSeg));
+                                                   Q2, s.ctr, k, (uint32_t)p.thread_deg_max, 0u);
     if (PROF && (rc = tm->end(g->stream))) return rc;
     if (PROF && (rc = tm->begin(g->stream, 3))) return rc;
     k_notify_big<PROF><<<g->sm_count * 8, kBlock, 0, g->stream>>>(g->ro, g->ci, s.C, W, s.S, Q2,

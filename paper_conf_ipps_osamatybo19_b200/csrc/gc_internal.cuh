@@ -117,6 +117,7 @@ struct RunParams {
     Keys keys;
     int32_t thread_deg_max = 8;
     int32_t hub_deg_min = 4096;
+    int32_t eval_big_min = 256;  // event mode: remaining scan length sent to a CTA
     int32_t batch_rounds = 0;
     int64_t max_rounds = 0;
 };
