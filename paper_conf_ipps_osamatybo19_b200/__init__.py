@@ -63,7 +63,9 @@ class gc_stats(ctypes.Structure):
                 ("ms", ctypes.c_double), ("frontier_sizes", ctypes.c_void_p),
                 ("frontier_cap", ctypes.c_int64), ("kernel_ms", ctypes.c_double * 4),
                 ("kernel_launches", ctypes.c_int64 * 4), ("kernel_bytes", ctypes.c_int64 * 4),
-                ("visits", ctypes.c_int64)]
+                ("visits", ctypes.c_int64), ("launch_us", ctypes.c_void_p),
+                ("launch_cap", ctypes.c_int64), ("round_stats", ctypes.c_void_p),
+                ("round_stats_cap", ctypes.c_int64)]
 
 
 _lib = None
@@ -142,6 +144,8 @@ class ColorStats:
     kernel_launches: list
     kernel_bytes: list
     visits: int
+    launch_us: list
+    round_stats: list
 
 
 class Graph:
@@ -169,7 +173,8 @@ class Graph:
 
     def color(self, seed: int = 1, variant: int = MAXMIN, out=None, *, flags: int = 0,
               mode: int = MODE_AUTO, batch_rounds: int = 0, thread_deg_max: int = 0,
-              hub_deg_min: int = 0, stats: bool = False, frontier_cap: int = 0):
+              hub_deg_min: int = 0, stats: bool = False, frontier_cap: int = 0,
+              trace_cap: int = 0):
         """Colour the graph.  `out`: int32 tensor/array of n entries on host or
         device (allocated on the host if None).  Returns (out, n_colors) or
         (out, n_colors, ColorStats) with stats=True."""
@@ -187,13 +192,21 @@ class Graph:
             fs = (ctypes.c_int64 * frontier_cap)()
             st.frontier_sizes = ctypes.cast(fs, ctypes.c_void_p)
             st.frontier_cap = frontier_cap
+        lu = rs = None
+        if trace_cap:
+            lu = (ctypes.c_float * (4 * trace_cap))()
+            rs = (ctypes.c_int64 * (4 * trace_cap))()
+            st.launch_us, st.launch_cap = ctypes.cast(lu, ctypes.c_void_p), 4 * trace_cap
+            st.round_stats, st.round_stats_cap = ctypes.cast(rs, ctypes.c_void_p), trace_cap
         r = _check(lib().gc_color_ex(self._h, ctypes.byref(o), _ptr(out, ("int32",)),
                                      ctypes.byref(st)))
         if stats:
             nk = list(fs[: min(frontier_cap, st.rounds)]) if fs is not None else []
             return out, r, ColorStats(st.mode_used, st.rounds, st.inner_iterations, st.n_colors,
                                       st.launches, st.ms, nk, list(st.kernel_ms),
-                                      list(st.kernel_launches), list(st.kernel_bytes), st.visits)
+                                      list(st.kernel_launches), list(st.kernel_bytes), st.visits,
+                                      list(lu[: min(4 * trace_cap, 4 * st.rounds + 8)]) if lu else [],
+                                      list(rs[: min(4 * trace_cap, 4 * st.rounds)]) if rs else [])
         return out, r
 
     def close(self) -> None:

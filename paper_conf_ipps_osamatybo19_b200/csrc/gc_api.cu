@@ -192,15 +192,21 @@ int ensure_nk(gc_graph *g, int64_t need) {
     Scratch &s = g->s;
     if (need <= s.nk_cap) return GC_OK;
     int64_t cap = std::max<int64_t>(need * 2, 1 << 12);
-    int64_t *nk = nullptr;
+    int64_t *nk = nullptr, *rstat = nullptr;
     GC_CUDA_TRY(cudaMalloc(&nk, sizeof(int64_t) * cap));
+    GC_CUDA_TRY(cudaMalloc(&rstat, sizeof(int64_t) * 4 * cap));
+    GC_CUDA_TRY(cudaMemsetAsync(rstat, 0, sizeof(int64_t) * 4 * cap, g->stream));
     if (s.nk) {
         GC_CUDA_TRY(cudaMemcpyAsync(nk, s.nk, sizeof(int64_t) * s.nk_cap, cudaMemcpyDeviceToDevice,
                                     g->stream));
+        GC_CUDA_TRY(cudaMemcpyAsync(rstat, s.rstat, sizeof(int64_t) * 4 * s.nk_cap,
+                                    cudaMemcpyDeviceToDevice, g->stream));
         GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
         cudaFree(s.nk);
+        cudaFree(s.rstat);
     }
     s.nk = nk;
+    s.rstat = rstat;
     s.nk_cap = cap;
     return GC_OK;
 }
@@ -293,6 +299,7 @@ static void free_scratch(Scratch &s) {
     cudaFree(s.Q2);
     cudaFree(s.ctr);
     cudaFree(s.nk);
+    cudaFree(s.rstat);
     cudaFree(s.bitmap);
     if (s.host_pinned) cudaFreeHost(s.host_pinned);
     s = Scratch();
@@ -540,6 +547,17 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
             stats->kernel_bytes[c] = prof.bytes[c];
         }
         stats->visits = prof.visits;
+        if (stats->launch_us && stats->launch_cap > 0) {
+            size_t m = std::min<size_t>((size_t)stats->launch_cap, prof.launch_us.size());
+            memcpy(stats->launch_us, prof.launch_us.data(), m * sizeof(float));
+        }
+        if (prof.on && stats->round_stats && stats->round_stats_cap > 0) {
+            int64_t m = std::min<int64_t>(std::min<int64_t>(stats->round_stats_cap, res.rounds + 1),
+                                          g->s.nk_cap);
+            if (m > 0)
+                GC_CUDA_TRY(cudaMemcpy(stats->round_stats, g->s.rstat, sizeof(int64_t) * 4 * m,
+                                       cudaMemcpyDeviceToHost));
+        }
         if (stats->frontier_sizes && stats->frontier_cap > 0 && !luby) {
             int64_t m = std::min<int64_t>(std::min<int64_t>(stats->frontier_cap, res.rounds),
                                           g->s.nk_cap);

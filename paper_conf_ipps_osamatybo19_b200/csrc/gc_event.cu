@@ -201,8 +201,9 @@ template <bool PROF>
 __global__ void __launch_bounds__(kBlock) k_eval(
     const int64_t *__restrict__ ro, const uint32_t *__restrict__ ci, uint32_t *C, uint2 *W,
     uint2 *P, const uint32_t *__restrict__ Din, uint32_t *__restrict__ Iout,
-    uint32_t *__restrict__ bigq, unsigned long long *ctr, int64_t *nk, int64_t nk_cap, uint32_t k,
-    uint32_t key, int dense, int64_t n, uint32_t thread_max, uint32_t big_min) {
+    uint32_t *__restrict__ bigq, unsigned long long *ctr, int64_t *nk, int64_t *rstat,
+    int64_t nk_cap, uint32_t k, uint32_t key, int dense, int64_t n, uint32_t thread_max,
+    uint32_t big_min) {
     const unsigned long long N = dense ? (unsigned long long)n : ctr[kD + k % 3];
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         ctr[kD + (k + 2) % 3] = 0;
@@ -210,7 +211,10 @@ __global__ void __launch_bounds__(kBlock) k_eval(
         ctr[kBE + (k + 1) % 3] = 0;
         ctr[kBN + k % 3] = 0;
         if ((int64_t)k < nk_cap) nk[k] = (int64_t)ctr[kRem];
-        if (PROF) ctr[kSumD] += N;
+        if (PROF) {
+            ctr[kSumD] += N;
+            if ((int64_t)k < nk_cap) rstat[4 * k] = (int64_t)N;
+        }
     }
     const uint32_t thresh = 2u * k;
     const unsigned lane = lane_id();
@@ -450,9 +454,14 @@ template <bool PROF>
 __global__ void __launch_bounds__(kBlock) k_notify_big(
     const int64_t *__restrict__ ro, const uint32_t *__restrict__ ci, const uint32_t *C,
     const uint2 *W, uint32_t *S, const uint2 *__restrict__ bigq, uint32_t *__restrict__ Dout,
-    unsigned long long *ctr, uint32_t k) {
+    unsigned long long *ctr, uint32_t k, int64_t *rstat, int64_t nk_cap) {
     const unsigned long long nitems = ctr[kBN + k % 3];
     unsigned long long *dcount = &ctr[kD + (k + 1) % 3];
+    if (PROF && blockIdx.x == 0 && threadIdx.x == 0 && (int64_t)k < nk_cap) {
+        rstat[4 * k + 1] = (int64_t)ctr[kI + k % 3];
+        rstat[4 * k + 2] = (int64_t)ctr[kBE + k % 3];
+        rstat[4 * k + 3] = (int64_t)nitems;
+    }
     const unsigned lane = lane_id();
     uint32_t nvis = 0;
     const unsigned long long warp0 = ((unsigned long long)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
@@ -494,7 +503,8 @@ int launch_round(gc_graph *g, const RunParams &p, uint32_t k, int grid, int grid
     int rc;
     if (PROF && (rc = tm->begin(g->stream, 0))) return rc;
     k_eval<PROF><<<dense ? grid_dense : grid, kBlock, 0, g->stream>>>(
-        g->ro, g->ci, s.C, W, P, D[k % 2], I, s.Q, s.ctr, s.nk, s.nk_cap, k, key, dense, g->n,
+        g->ro, g->ci, s.C, W, P, D[k % 2], I, s.Q, s.ctr, s.nk, s.rstat, s.nk_cap, k, key, dense,
+        g->n,
         (uint32_t)p.thread_deg_max, (uint32_t)p.eval_big_min);
     if (PROF && (rc = tm->end(g->stream))) return rc;
     if (PROF && (rc = tm->begin(g->stream, 1))) return rc;
@@ -508,7 +518,8 @@ int launch_round(gc_graph *g, const RunParams &p, uint32_t k, int grid, int grid
     if (PROF && (rc = tm->end(g->stream))) return rc;
     if (PROF && (rc = tm->begin(g->stream, 3))) return rc;
     k_notify_big<PROF><<<g->sm_count * 8, kBlock, 0, g->stream>>>(g->ro, g->ci, s.C, W, s.S, Q2,
-                                                                  D[(k + 1) % 2], s.ctr, k);
+                                                                  D[(k + 1) % 2], s.ctr, k,
+                                                                  s.rstat, s.nk_cap);
     if (PROF && (rc = tm->end(g->stream))) return rc;
     return GC_OK;
 }

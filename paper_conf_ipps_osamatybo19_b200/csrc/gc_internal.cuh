@@ -53,6 +53,7 @@ struct Scratch {
     unsigned long long *ctr = nullptr;  // device counters (see gc_sweep.cu)
     int64_t *nk = nullptr;        // per-round frontier sizes (stats), cap nk_cap
     int64_t nk_cap = 0;
+    int64_t *rstat = nullptr;     // PROF: 4 counters per round (cap nk_cap)
     uint32_t *bitmap = nullptr;   // colour-count bitmap
     int64_t bitmap_words = 0;
     int64_t *host_pinned = nullptr;  // pinned readback area
@@ -98,6 +99,7 @@ struct Profile {
     int64_t launches[4] = {0, 0, 0, 0};
     int64_t bytes[4] = {0, 0, 0, 0};
     int64_t visits = 0;
+    std::vector<float> launch_us;   // every timed launch, in order
 };
 
 // Pool of CUDA events bracketing individual launches in profile mode.

@@ -313,6 +313,7 @@ int EventTimer::drain(Profile *p) {
         GC_CUDA_TRY(cudaEventElapsedTime(&ms, ev[i], ev[i + 1]));
         p->ms[cls[i / 2]] += ms;
         p->launches[cls[i / 2]] += 1;
+        p->launch_us.push_back(1e3f * ms);
     }
     used = 0;
     return GC_OK;

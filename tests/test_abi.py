@@ -54,7 +54,7 @@ def test_library_is_sm100a_only(libgc):
 def test_struct_layouts_match_header(libgc):
     # gc_options / gc_stats sizes as compiled in C (see include/gc.h)
     assert ctypes.sizeof(gcb.gc_options) == 4 + 4 + 8 + 4 + 4 + 4 + 4 + 4 + 28
-    assert ctypes.sizeof(gcb.gc_stats) == 4 + 4 + 8 * 4 + 8 + 8 + 8 + 8 * 4 * 3 + 8
+    assert ctypes.sizeof(gcb.gc_stats) == 4 + 4 + 8 * 4 + 8 + 8 + 8 + 8 * 4 * 3 + 8 + 8 * 4
 
 
 def test_fails_loudly_without_gpu(libgc):

@@ -1,0 +1,63 @@
+"""Per-round profile of one colouring (GC_PROFILE): kernel durations per round
+and queue sizes, summarised in buckets.  Writes JSON to --out.
+
+    python tools/round_profile.py --scale 24 [--mode event] --out gpurun_out/rounds.json
+"""
+import argparse
+import json
+import os
+import sys
+
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+
+import torch  # noqa: E402
+
+import graphgen as G  # noqa: E402
+import paper_conf_ipps_osamatybo19_b200 as gcb  # noqa: E402
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--scale", type=int, default=24)
+    ap.add_argument("--mode", default="event")
+    ap.add_argument("--out", default="gpurun_out/rounds.json")
+    a = ap.parse_args()
+    g = G.rmat(a.scale, 16, seed=1, device="cuda")
+    mode = {"event": gcb.MODE_EVENT, "sweep": gcb.MODE_SWEEP}[a.mode]
+    out = torch.empty(g.n, dtype=torch.int32, device="cuda")
+    with gcb.Graph(g.n, g.row_offsets, g.col_indices, flags=gcb.BORROW_DEVICE) as h:
+        h.color(1, gcb.MAXMIN, out, mode=mode)
+        _, k, st = h.color(1, gcb.MAXMIN, out, mode=mode, flags=gcb.PROFILE, stats=True,
+                           trace_cap=1 << 15)
+    R = st.rounds
+    per = 4 if mode == gcb.MODE_EVENT else 2
+    lu = st.launch_us
+    rows = []
+    for r in range(R):
+        t = lu[per * r: per * r + per]
+        rs = st.round_stats[4 * r: 4 * r + 4]
+        rows.append({"k": r, "us": t, "stats": rs})
+    buckets = [(0, 1), (1, 2), (2, 10), (10, 100), (100, 500), (500, 1000), (1000, 2000),
+               (2000, R)]
+    summ = []
+    for lo, hi in buckets:
+        sel = rows[lo:min(hi, R)]
+        if not sel:
+            continue
+        tot = [sum(x["us"][c] for x in sel) for c in range(per)]
+        st4 = [sum(x["stats"][c] for x in sel) for c in range(4)]
+        summ.append({"rounds": [lo, min(hi, R)], "us_by_class": tot, "us_total": sum(tot),
+                     "stat_sums": st4, "us_per_round": sum(tot) / len(sel)})
+    res = {"scale": a.scale, "mode": a.mode, "rounds": R, "n_colors": k, "ms": st.ms,
+           "kernel_ms": st.kernel_ms, "buckets": summ,
+           "top_rounds": sorted(rows, key=lambda x: -sum(x["us"]))[:25]}
+    os.makedirs(os.path.dirname(a.out) or ".", exist_ok=True)
+    with open(a.out, "w") as f:
+        json.dump(res, f, indent=1)
+    for b in summ:
+        print(json.dumps(b))
+    print("top:", [(x["k"], [round(u, 1) for u in x["us"]], x["stats"]) for x in res["top_rounds"][:12]])
+
+
+if __name__ == "__main__":
+    main()
