@@ -44,7 +44,7 @@ def parse():
     ap.add_argument("--scale", type=int, default=0, help="R-MAT scale (default 24+log2 N)")
     ap.add_argument("--variant", default="maxmin", choices=["maxmin", "luby", "multihash"])
     ap.add_argument("--hashes", type=int, default=4)
-    ap.add_argument("--mode", default="auto", choices=["auto", "sweep", "event"])
+    ap.add_argument("--mode", default="auto", choices=["auto", "sweep", "event", "event-multi"])
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-profile", action="store_true")
@@ -213,7 +213,8 @@ def main():
     scale = args.scale or (24 + int(round(math.log2(max(1, world)))))
     variant = {"maxmin": gcb.MAXMIN, "luby": gcb.LUBY_MIS,
                "multihash": gcb.MULTIHASH(args.hashes)}[args.variant]
-    mode = {"auto": gcb.MODE_AUTO, "sweep": gcb.MODE_SWEEP, "event": gcb.MODE_EVENT}[args.mode]
+    mode = {"auto": gcb.MODE_AUTO, "sweep": gcb.MODE_SWEEP, "event": gcb.MODE_EVENT,
+            "event-multi": gcb.MODE_EVENT_MULTI}[args.mode]
 
     t0 = time.time()
     if world > 1:
@@ -267,7 +268,8 @@ def main():
         total_ms = float(t.item())
     ms_per = total_ms / args.steps
     value = nnz_global * args.steps / (total_ms / 1e3) / 1e9
-    mode_used = {1: "sweep", 2: "event"}.get(st.mode_used, str(st.mode_used))
+    mode_used = {1: "sweep", 2: "event (persistent)", 3: "event (multi-kernel)"}.get(
+        st.mode_used, str(st.mode_used))
 
     # ---- roofline of the dominant kernel: a profiled pass (GC_PROFILE brackets
     # every sweep launch with events on this stream); separate from the timed steps
@@ -277,9 +279,13 @@ def main():
         torch.cuda.synchronize()
         peak, peak_src = measured_peaks()
         cls = max(range(4), key=lambda c: sp.kernel_ms[c])
-        names = ({0: "k_eval", 1: "k_eval_big", 2: "k_notify", 3: "k_notify_big"}
-                 if sp.mode_used == gcb.MODE_EVENT else
-                 {0: "k_sweep", 1: "k_hub", 2: "other", 3: "other"})
+        names = {gcb.MODE_EVENT: {0: "k_event_persistent", 1: "phase P1 eval",
+                                  2: "phase P1b+P2 long scans", 3: "phase P3 notify"},
+                 gcb.MODE_EVENT_MULTI: {0: "k_eval", 1: "k_eval_big", 2: "k_notify",
+                                        3: "k_notify_big"},
+                 gcb.MODE_SWEEP: {0: "k_sweep", 1: "k_hub", 2: "other", 3: "other"}}[sp.mode_used]
+        if sp.mode_used == gcb.MODE_EVENT:
+            cls = 0  # one persistent launch; classes 1-3 are its phases (globaltimer)
         name = names[cls]
         kms, kl, kb = sp.kernel_ms[cls], sp.kernel_launches[cls], sp.kernel_bytes[cls]
         achieved = (kb / 1e9) / (kms / 1e3) if kms > 0 else 0.0
@@ -291,7 +297,7 @@ def main():
                 "visits": sp.visits, "profiled_ms": sp.ms,
                 "classes": {names[c]: {"ms": sp.kernel_ms[c], "launches": sp.kernel_launches[c],
                                        "bytes": sp.kernel_bytes[c]} for c in range(4)
-                            if sp.kernel_launches[c]}}
+                            if sp.kernel_ms[c] > 0}}
 
     # ---- end to end through the C ABI with host buffers
     e2e = None

@@ -92,7 +92,9 @@ typedef enum gc_status {
                             with early exit (the paper's ComputeOp shape) */
 #define GC_MODE_EVENT 2  /* work-efficient: per-vertex witnesses + resume
                             cursors; only neighbours of newly coloured
-                            vertices are re-evaluated */
+                            vertices are re-evaluated; all
+                            rounds in one persistent cooperative kernel */
+#define GC_MODE_EVENT_MULTI 3 /* the same method, 4 kernel launches per round */
 
 typedef struct gc_graph gc_graph;
 
@@ -112,7 +114,7 @@ typedef struct gc_options {
 /* Statistics filled by gc_color_ex (optional). */
 typedef struct gc_stats {
     uint32_t struct_size;     /* sizeof(gc_stats) */
-    int32_t mode_used;        /* GC_MODE_SWEEP or GC_MODE_EVENT */
+    int32_t mode_used;        /* GC_MODE_SWEEP, GC_MODE_EVENT or GC_MODE_EVENT_MULTI */
     int64_t rounds;           /* R: rounds (max-min / multi-hash) or colours (Luby) */
     int64_t inner_iterations; /* Luby: Alg.3 do-while iterations; else == rounds */
     int64_t n_colors;         /* distinct colours */

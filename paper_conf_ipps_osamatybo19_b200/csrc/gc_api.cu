@@ -232,6 +232,8 @@ int ensure_scratch(gc_graph *g, bool need_event, bool need_luby) {
         GC_CUDA_TRY(cudaMalloc(&s.Q, nn * 4));
         // long-row notify items (u, segment): at most n + nnz/128 per round
         GC_CUDA_TRY(cudaMalloc(&s.Q2, (nn + (size_t)g->nnz / 128 + 1) * 8));
+        GC_CUDA_TRY(cudaMalloc(&s.Q3, (nn + (size_t)g->nnz / 128 + 1) * 8));
+        GC_CUDA_TRY(cudaMalloc(&s.LS, nn * 32));
     }
     return GC_OK;
 }
@@ -297,6 +299,8 @@ static void free_scratch(Scratch &s) {
     cudaFree(s.P);
     cudaFree(s.Q);
     cudaFree(s.Q2);
+    cudaFree(s.Q3);
+    cudaFree(s.LS);
     cudaFree(s.ctr);
     cudaFree(s.nk);
     cudaFree(s.rstat);
@@ -470,7 +474,7 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
         set_error("gc_color_ex: unknown variant");
         return GC_ERR_INVALID_ARG;
     }
-    if (o->mode < GC_MODE_AUTO || o->mode > GC_MODE_EVENT) {
+    if (o->mode < GC_MODE_AUTO || o->mode > GC_MODE_EVENT_MULTI) {
         set_error("gc_color_ex: unknown mode");
         return GC_ERR_INVALID_ARG;
     }
@@ -481,9 +485,9 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     int mode = o->mode;
     if (mode == GC_MODE_AUTO) mode = GC_MODE_EVENT;
     if (luby) mode = GC_MODE_SWEEP;
-    if (mode == GC_MODE_EVENT && H != 1) mode = GC_MODE_SWEEP;
+    if (mode != GC_MODE_SWEEP && H != 1) mode = GC_MODE_SWEEP;
 
-    int rc = ensure_scratch(g, mode == GC_MODE_EVENT, luby);
+    int rc = ensure_scratch(g, mode != GC_MODE_SWEEP, luby);
     if (rc) return rc;
     RunParams p;
     p.H = H;
@@ -505,6 +509,8 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     if (luby)
         rc = run_luby(g, p, &res);
     else if (mode == GC_MODE_EVENT)
+        rc = run_persistent_maxmin(g, p, &res);
+    else if (mode == GC_MODE_EVENT_MULTI)
         rc = run_event_maxmin(g, p, &res);
     else
         rc = run_sweep_maxmin(g, p, &res);

@@ -46,7 +46,9 @@ struct Scratch {
     uint32_t *F[2] = {nullptr, nullptr};  // frontiers (vertex ids)
     uint32_t *hub = nullptr;      // per-round hub work list / event: coloured list I_k
     uint32_t *Q = nullptr;        // event mode: long-scan queue
-    uint32_t *Q2 = nullptr;       // event mode: long-row notify queue
+    uint32_t *Q2 = nullptr;       // event mode: long-row notify / long-scan segment queue
+    uint32_t *Q3 = nullptr;       // persistent event mode: notify segment queue
+    void *LS = nullptr;           // persistent event mode: long-scan slots (32 B each)
     uint32_t *S = nullptr;        // Luby inner-loop state / event stamps
     uint32_t *W = nullptr;        // event mode: witness pairs (2 per vertex)
     uint32_t *P = nullptr;        // event mode: resume cursors (2 per vertex)
@@ -133,6 +135,7 @@ struct RunResult {
 int ensure_scratch(gc_graph *g, bool need_event, bool need_luby);
 int run_sweep_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int run_event_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
+int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int run_luby(gc_graph *g, const RunParams &p, RunResult *r);
 int64_t count_colors_device(gc_graph *g, const uint32_t *C, int64_t n, bool compact,
                             uint32_t *C_inout, int64_t *launches);

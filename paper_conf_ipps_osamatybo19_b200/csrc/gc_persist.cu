@@ -1,0 +1,504 @@
+// gc_persist.cu -- EVENT mode as ONE persistent cooperative kernel that runs
+// every round of the max-min colouring (Alg.1 + Alg.5, P:L102-113,
+// P:L506-556; H = 1) with grid-wide barriers instead of kernel boundaries.
+//
+// The method per round is the witness/resume scheme of gc_event.cu; this file
+// only changes how the work of a round is scheduled on the 148 SMs:
+//   P1  evaluate D_k: one lane per vertex (round 0 and large D_k: scan a
+//       window of kLaneWin entries, unresolved rows go to WQ) or one warp per
+//       vertex (scan a kWarpWin window, unresolved rows become long scans);
+//   P1b WQ: one warp per vertex, same as the warp path of P1;
+//   P2  long scans split into kSeg-entry segments over all warps; each segment
+//       atomicMin's its first hi / lo hit into the scan's slot, and the warp
+//       finishing the last segment settles the vertex (first-hit semantics are
+//       kept, so the cursor invariant holds);
+//   P3  notify: rows of vertices coloured in this round -- short rows one lane
+//       each, long rows as kNotifySeg-entry segments over all warps -- wake the
+//       uncoloured neighbours that used the coloured vertex as a witness.
+// A phase whose queue is empty is skipped (its barrier too): the decision is
+// taken after a barrier from device counters, so it is grid-uniform.
+// The host launches one kernel per colouring; per-round sizes land in nk[].
+#include <cooperative_groups.h>
+
+#include "gc_event_common.cuh"
+
+namespace cg = cooperative_groups;
+
+namespace gc {
+
+int fill_u32(uint32_t *p, uint32_t val, int64_t n, cudaStream_t st);
+int ensure_nk(gc_graph *g, int64_t need);
+
+namespace {
+
+using namespace ev;
+
+constexpr int kThreads = 512;
+constexpr int kLaneWin = 8;      // entries a lane scans before handing off
+constexpr int kWarpWin = 256;    // entries a warp scans before splitting
+constexpr int kSeg = 256;        // entries per long-scan segment (8 per lane)
+constexpr int kNotifySeg = 128;  // entries per notify segment (4 per lane)
+constexpr int kLaneNotify = 32;  // rows up to this length are notified by one lane
+
+// counter layout: two sets of 8 (by round parity) at ctr[24..39]
+enum : int { cD = 0, cWQ = 1, cSQ = 2, cLS = 3, cNQS = 4, cNQ = 5, cI = 6 };
+enum : int {
+    kSet = 24,
+    kRem = 40,
+    kVisE = 41,
+    kVisS = 42,
+    kVisN = 43,
+    kSumD = 44,
+    kRounds = 45,
+    kPhaseNs = 50  // [50..53] PROF: ns spent in P1, P1b+P2, P3, barriers
+};
+
+struct LongScan {   // one slot per long scan of a round (32 B)
+    uint32_t v;
+    uint32_t ticket;  // segments still outstanding
+    uint32_t minH;    // first hi hit, relative to the row start (kNone: none)
+    uint32_t minL;
+    uint32_t need;    // bit 0: hi still searched, bit 1: lo
+    uint32_t sh, sl;  // search starts (relative)
+    uint32_t base;    // relative start of segment 0
+};
+
+struct Args {
+    const int64_t *ro;
+    const uint32_t *ci;
+    uint32_t *C;
+    uint2 *W;
+    uint2 *P;
+    uint32_t *S;
+    uint32_t *D[2];
+    uint32_t *WQ;
+    uint2 *SQ;
+    LongScan *LS;
+    uint32_t *NQS;
+    uint2 *NQ;
+    unsigned long long *ctr;
+    int64_t *nk;
+    int64_t *rstat;
+    int64_t nk_cap;
+    int64_t n;
+    uint32_t key;
+    uint32_t max_rounds;
+};
+
+__device__ __forceinline__ unsigned long long gtimer() {
+    unsigned long long t;
+    asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+    return t;
+}
+
+// Enqueue the notification work of lanes whose vertex was just coloured
+// (whole warp converged).  Short rows -> NQS (one lane each); long rows ->
+// NQ segments.
+__device__ __forceinline__ void enqueue_notify(const Args &a, unsigned long long *cs, bool colored,
+                                               uint32_t u, int64_t deg) {
+    const bool shortrow = colored && deg <= kLaneNotify;
+    warp_append(shortrow, u, a.NQS, &cs[cNQS]);
+    unsigned lm = __ballot_sync(kFull, colored && !shortrow);
+    while (lm) {  // long rows: the whole warp writes the segment items
+        const int src = __ffs(lm) - 1;
+        lm &= lm - 1;
+        const uint32_t uu = __shfl_sync(kFull, u, src);
+        const int64_t dg = __shfl_sync(kFull, deg, src);
+        const uint32_t nseg = (uint32_t)((dg + kNotifySeg - 1) / kNotifySeg);
+        unsigned long long b = 0;
+        if (lane_id() == 0) b = atomicAdd(&cs[cNQ], (unsigned long long)nseg);
+        b = __shfl_sync(kFull, b, 0);
+        for (uint32_t q = lane_id(); q < nseg; q += 32) a.NQ[b + q] = make_uint2(uu, q);
+    }
+    const unsigned m = __ballot_sync(kFull, colored);
+    if (m && lane_id() == (unsigned)(__ffs(m) - 1)) atomicAdd(&cs[cI], (unsigned long long)__popc(m));
+}
+
+// Whole-warp evaluation of one vertex of D_k (warp-uniform arguments): scan a
+// window; resolved -> settle; otherwise open a long scan (P2).
+template <bool PROF>
+__device__ __forceinline__ void eval_warp(const Args &a, unsigned long long *cs, uint32_t v,
+                                          uint32_t k, bool dense, uint32_t &nvis) {
+    const uint32_t thresh = 2u * k;
+    const unsigned lane = lane_id();
+    const int64_t rs = a.ro[v], re = a.ro[v + 1];
+    const Resume r = resume_of(v, rs, dense, a.W, a.P, a.C, thresh);
+    if (!r.need_hi && !r.need_lo) return;
+    int64_t s = r.need_hi ? r.sh : re;
+    if (r.need_lo && r.sl < s) s = r.sl;
+    const int64_t lim = min(re, s + (int64_t)kWarpWin);
+    Found f;
+    uint32_t vis = 0;
+    warp_search(a.ci, a.C, thresh, a.key, weight_mix(v ^ a.key), r.need_hi, r.need_lo, r.sh, r.sl,
+                lim, f, vis);
+    if (PROF) nvis += vis;
+    const bool miss_hi = r.need_hi && f.hpos < 0;
+    const bool miss_lo = r.need_lo && f.lpos < 0;
+    if (lim < re && (miss_hi || miss_lo)) {
+        // long scan of [lim, re) for the missing sides
+        const uint32_t nseg = (uint32_t)((re - lim + kSeg - 1) / kSeg);
+        unsigned long long slot = 0, b = 0;
+        if (lane == 0) {
+            slot = atomicAdd(&cs[cLS], 1ull);
+            LongScan L;
+            L.v = v;
+            L.ticket = nseg;
+            L.minH = f.hpos >= 0 ? (uint32_t)(f.hpos - rs) : kNone;
+            L.minL = f.lpos >= 0 ? (uint32_t)(f.lpos - rs) : kNone;
+            L.need = (miss_hi ? 1u : 0u) | (miss_lo ? 2u : 0u);
+            L.sh = (uint32_t)(r.sh - rs);
+            L.sl = (uint32_t)(r.sl - rs);
+            L.base = (uint32_t)(lim - rs);
+            a.LS[slot] = L;
+            b = atomicAdd(&cs[cSQ], (unsigned long long)nseg);
+        }
+        slot = __shfl_sync(kFull, slot, 0);
+        b = __shfl_sync(kFull, b, 0);
+        for (uint32_t q = lane; q < nseg; q += 32) a.SQ[b + q] = make_uint2((uint32_t)slot, q);
+        return;
+    }
+    bool colored = false;
+    if (lane == 0) colored = settle(v, rs, r, f, k, a.C, a.W, a.P);
+    colored = __shfl_sync(kFull, colored, 0);
+    enqueue_notify(a, cs, colored && lane == 0, v, re - rs);
+}
+
+// One kSeg-entry segment of a long scan (whole warp).
+template <bool PROF>
+__device__ __forceinline__ void scan_segment(const Args &a, unsigned long long *cs, uint2 item,
+                                             uint32_t k, bool dense, uint32_t &nvis) {
+    const unsigned lane = lane_id();
+    const uint32_t thresh = 2u * k;
+    LongScan *L = &a.LS[item.x];
+    const uint32_t v = L->v;
+    const uint32_t need = L->need;
+    const int64_t rs = a.ro[v], re = a.ro[v + 1];
+    const int64_t e0 = rs + (int64_t)L->base + (int64_t)item.y * kSeg;
+    const int64_t e1 = min(re, e0 + (int64_t)kSeg);
+    const uint32_t pv = weight_mix(v ^ a.key);
+    // skip when every needed side already has a hit before this segment
+    const uint32_t curH = *(volatile uint32_t *)&L->minH, curL = *(volatile uint32_t *)&L->minL;
+    const uint32_t rel0 = (uint32_t)(e0 - rs);
+    const bool want_hi = (need & 1u) && !(curH != kNone && curH < rel0);
+    const bool want_lo = (need & 2u) && !(curL != kNone && curL < rel0);
+    if (want_hi || want_lo) {
+        uint32_t u[kSeg / 32], c[kSeg / 32];
+#pragma unroll
+        for (int q = 0; q < kSeg / 32; ++q) {
+            const int64_t e = e0 + q * 32 + lane;
+            u[q] = e < e1 ? a.ci[e] : 0u;
+        }
+#pragma unroll
+        for (int q = 0; q < kSeg / 32; ++q) {
+            const int64_t e = e0 + q * 32 + lane;
+            c[q] = e < e1 ? a.C[u[q]] : 0u;
+        }
+        uint32_t rh = kNone, rl = kNone;
+#pragma unroll
+        for (int q = 0; q < kSeg / 32; ++q) {
+            const int64_t e = e0 + q * 32 + lane;
+            if (e < e1 && c[q] >= thresh) {
+                const uint32_t pu = weight_mix(u[q] ^ a.key);
+                const uint32_t rel = (uint32_t)(e - rs);
+                if (want_hi && rel >= L->sh && pu > pv) rh = min(rh, rel);
+                if (want_lo && rel >= L->sl && pu < pv) rl = min(rl, rel);
+            }
+        }
+        if (PROF) {
+            const int64_t cnt = e1 - e0 - (int64_t)lane;  // this lane's entries in the segment
+            nvis += cnt > 0 ? (uint32_t)((cnt + 31) / 32) : 0u;
+        }
+        rh = __reduce_min_sync(kFull, rh);
+        rl = __reduce_min_sync(kFull, rl);
+        if (lane == 0) {
+            if (rh != kNone) atomicMin(&L->minH, rh);
+            if (rl != kNone) atomicMin(&L->minL, rl);
+        }
+    }
+    bool last = false;
+    if (lane == 0) {
+        __threadfence();
+        last = atomicSub(&L->ticket, 1u) == 1u;
+    }
+    last = __shfl_sync(kFull, last, 0);
+    if (!last) return;
+    // the warp that finished the last segment settles v
+    bool colored = false;
+    if (lane == 0) {
+        __threadfence();
+        const uint32_t mH = atomicAdd(&L->minH, 0u), mL = atomicAdd(&L->minL, 0u);
+        const Resume r = resume_of(v, rs, dense, a.W, a.P, a.C, thresh);
+        Found f;
+        if (mH != kNone) {
+            f.hpos = rs + mH;
+            f.hw = a.ci[f.hpos];
+        }
+        if (mL != kNone) {
+            f.lpos = rs + mL;
+            f.lw = a.ci[f.lpos];
+        }
+        colored = settle(v, rs, r, f, k, a.C, a.W, a.P);
+    }
+    colored = __shfl_sync(kFull, colored, 0);
+    enqueue_notify(a, cs, colored && lane == 0, v, re - rs);
+}
+
+template <bool PROF>
+__global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
+    cg::grid_group grid = cg::this_grid();
+    const unsigned lane = lane_id();
+    const unsigned long long gtid = (unsigned long long)blockIdx.x * blockDim.x + threadIdx.x;
+    const unsigned long long nthreads = (unsigned long long)gridDim.x * blockDim.x;
+    const unsigned long long gwarp = gtid >> 5, nwarps = nthreads >> 5;
+    unsigned long long rem = a.ctr[kRem];
+    uint32_t nvisE = 0, nvisS = 0, nvisN = 0;
+    unsigned long long t0 = 0, tacc[4] = {0, 0, 0, 0};
+    uint32_t k = 0;
+    for (;; ++k) {
+        unsigned long long *cs = a.ctr + kSet + 8 * (k & 1);
+        unsigned long long *cn = a.ctr + kSet + 8 * ((k + 1) & 1);
+        if (gtid == 0 && (int64_t)k < a.nk_cap) a.nk[k] = (int64_t)rem;
+        if (rem == 0 || k >= a.max_rounds) break;  // uniform: rem is computed identically
+        const bool dense = k == 0;
+        const unsigned long long N = dense ? (unsigned long long)a.n : cs[cD];
+        if (gtid == 0) {
+            for (int i = 0; i < 8; ++i) cn[i] = 0;
+            if (PROF) {
+                a.ctr[kSumD] += N;
+                if ((int64_t)k < a.nk_cap) a.rstat[4 * k] = (int64_t)N;
+                t0 = gtimer();
+            }
+        }
+        const uint32_t *Din = a.D[k & 1];
+        uint32_t *Dout = a.D[(k + 1) & 1];
+        const uint32_t thresh = 2u * k;
+        // ------------------------------------------------------------ P1
+        if (dense || N > 4 * nwarps) {
+            for (unsigned long long base = gwarp * 32; base < N; base += nthreads) {
+                const unsigned long long idx = base + lane;
+                const bool valid = idx < N;
+                uint32_t v = 0;
+                int64_t rs = 0, re = 0;
+                Resume r{false, false, 0, 0};
+                if (valid) {
+                    v = dense ? (uint32_t)idx : Din[idx];
+                    rs = a.ro[v];
+                    re = a.ro[v + 1];
+                    r = resume_of(v, rs, dense, a.W, a.P, a.C, thresh);
+                }
+                const bool work = valid && (r.need_hi || r.need_lo);
+                int64_t s = r.need_hi ? r.sh : re;
+                if (r.need_lo && r.sl < s) s = r.sl;
+                const int64_t lim = min(re, s + (int64_t)kLaneWin);
+                Found f;
+                uint32_t vis = 0;
+                if (work)
+                    lane_search(a.ci, a.C, thresh, a.key, weight_mix(v ^ a.key), r.need_hi,
+                                r.need_lo, r.sh, r.sl, lim, f, vis);
+                if (PROF) nvisE += vis;
+                const bool unresolved =
+                    work && lim < re && ((r.need_hi && f.hpos < 0) || (r.need_lo && f.lpos < 0));
+                bool colored = false;
+                if (work && !unresolved) colored = settle(v, rs, r, f, k, a.C, a.W, a.P);
+                warp_append(unresolved, v, a.WQ, &cs[cWQ]);
+                enqueue_notify(a, cs, colored, v, re - rs);
+            }
+        } else {
+            for (unsigned long long i = gwarp; i < N; i += nwarps)
+                eval_warp<PROF>(a, cs, Din[i], k, false, nvisE);
+        }
+        grid.sync();
+        if (PROF && gtid == 0) {
+            unsigned long long t = gtimer();
+            tacc[0] += t - t0;
+            t0 = t;
+        }
+        // ----------------------------------------------------------- P1b
+        const unsigned long long nwq = cs[cWQ];
+        if (nwq) {
+            for (unsigned long long i = gwarp; i < nwq; i += nwarps)
+                eval_warp<PROF>(a, cs, a.WQ[i], k, dense, nvisE);
+            grid.sync();
+        }
+        // ------------------------------------------------------------ P2
+        const unsigned long long nsq = cs[cSQ];
+        if (nsq) {
+            for (unsigned long long i = gwarp; i < nsq; i += nwarps)
+                scan_segment<PROF>(a, cs, a.SQ[i], k, dense, nvisS);
+            grid.sync();
+        }
+        if (PROF && gtid == 0) {
+            unsigned long long t = gtimer();
+            tacc[1] += t - t0;
+            t0 = t;
+        }
+        // ------------------------------------------------------------ P3
+        const unsigned long long ncol = cs[cI];
+        const unsigned long long nqs = cs[cNQS], nq = cs[cNQ];
+        unsigned long long *dcount = &cn[cD];
+        for (unsigned long long base = gwarp * 32; base < nqs; base += nthreads) {
+            const unsigned long long idx = base + lane;
+            if (idx < nqs) {
+                const uint32_t u = a.NQS[idx];
+                const int64_t rs = a.ro[u], re = a.ro[u + 1];
+                for (int64_t e = rs; e < re; ++e) {
+                    const uint32_t w = a.ci[e];
+                    if (wake(w, u, k, a.C, a.W, a.S)) Dout[atomicAdd(dcount, 1ull)] = w;
+                }
+                if (PROF) nvisN += (uint32_t)(re - rs);
+            }
+        }
+        for (unsigned long long it = gwarp; it < nq; it += nwarps) {
+            const uint2 item = a.NQ[it];
+            const uint32_t u = item.x;
+            const int64_t rs = a.ro[u] + (int64_t)item.y * kNotifySeg;
+            const int64_t re = min(a.ro[u + 1], rs + (int64_t)kNotifySeg);
+            uint32_t w[kNotifySeg / 32];
+#pragma unroll
+            for (int q = 0; q < kNotifySeg / 32; ++q) {
+                const int64_t e = rs + q * 32 + lane;
+                w[q] = e < re ? a.ci[e] : kNone;
+            }
+#pragma unroll
+            for (int q = 0; q < kNotifySeg / 32; ++q) {
+                const bool wk = w[q] != kNone && wake(w[q], u, k, a.C, a.W, a.S);
+                warp_append(wk, w[q], Dout, dcount);
+            }
+            if (PROF && lane == 0) nvisN += (uint32_t)(re - rs);
+        }
+        if (PROF && gtid == 0 && (int64_t)k < a.nk_cap) {
+            a.rstat[4 * k + 1] = (int64_t)ncol;
+            a.rstat[4 * k + 2] = (int64_t)cs[cLS];
+            a.rstat[4 * k + 3] = (int64_t)nq;
+        }
+        rem -= ncol;
+        grid.sync();
+        if (PROF && gtid == 0) {
+            unsigned long long t = gtimer();
+            tacc[2] += t - t0;
+            t0 = t;
+        }
+    }
+    if (gtid == 0) {
+        a.ctr[kRem] = rem;
+        a.ctr[kRounds] = k;
+        if (PROF)
+            for (int i = 0; i < 4; ++i) a.ctr[kPhaseNs + i] = tacc[i];
+    }
+    if (PROF) {
+        const unsigned e = __reduce_add_sync(kFull, nvisE);
+        const unsigned s = __reduce_add_sync(kFull, nvisS);
+        const unsigned q = __reduce_add_sync(kFull, nvisN);
+        if (lane == 0) {
+            if (e) atomicAdd(&a.ctr[kVisE], (unsigned long long)e);
+            if (s) atomicAdd(&a.ctr[kVisS], (unsigned long long)s);
+            if (q) atomicAdd(&a.ctr[kVisN], (unsigned long long)q);
+        }
+    }
+}
+
+template <bool PROF>
+int launch(gc_graph *g, Args &a, int *blocks_out) {
+    int per_sm = 0;
+    GC_CUDA_TRY(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_event_persistent<PROF>,
+                                                              kThreads, 0));
+    if (per_sm < 1) {
+        set_error("persistent event kernel cannot be resident");
+        return GC_ERR_CUDA;
+    }
+    const int blocks = per_sm * g->sm_count;
+    void *args[] = {&a};
+    GC_CUDA_TRY(cudaLaunchCooperativeKernel((void *)k_event_persistent<PROF>, blocks, kThreads, args,
+                                            0, g->stream));
+    *blocks_out = blocks;
+    return GC_OK;
+}
+
+}  // namespace
+
+int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
+    Scratch &s = g->s;
+    const int64_t n = g->n;
+    r->rounds = r->inner = r->launches = 0;
+    if (n == 0) return GC_OK;
+    int rc = fill_u32(s.C, GC_UNC, n, g->stream);  // Alg.5 L5
+    if (rc) return rc;
+    GC_CUDA_TRY(cudaMemsetAsync(s.S, 0, sizeof(uint32_t) * (size_t)n, g->stream));
+    GC_CUDA_TRY(cudaMemsetAsync(s.ctr, 0, 56 * sizeof(unsigned long long), g->stream));
+    const unsigned long long rem = (unsigned long long)n;
+    GC_CUDA_TRY(cudaMemcpyAsync(s.ctr + kRem, &rem, sizeof(rem), cudaMemcpyHostToDevice, g->stream));
+    const int64_t max_rounds = std::min<int64_t>(p.max_rounds, 0xFFFFFFF0ll);
+    rc = ensure_nk(g, std::min<int64_t>(std::min<int64_t>(n + 2, max_rounds + 2), 1 << 20));
+    if (rc) return rc;
+    Args a;
+    a.ro = g->ro;
+    a.ci = g->ci;
+    a.C = s.C;
+    a.W = reinterpret_cast<uint2 *>(s.W);
+    a.P = reinterpret_cast<uint2 *>(s.P);
+    a.S = s.S;
+    a.D[0] = s.F[0];
+    a.D[1] = s.F[1];
+    a.WQ = s.hub;
+    a.SQ = reinterpret_cast<uint2 *>(s.Q2);
+    a.LS = reinterpret_cast<LongScan *>(s.LS);
+    a.NQS = s.Q;
+    a.NQ = reinterpret_cast<uint2 *>(s.Q3);
+    a.ctr = s.ctr;
+    a.nk = s.nk;
+    a.rstat = s.rstat;
+    a.nk_cap = s.nk_cap;
+    a.n = n;
+    a.key = p.keys.k[0];
+    a.max_rounds = (uint32_t)max_rounds;
+    const bool prof = p.prof && p.prof->on;
+    cudaEvent_t e0 = nullptr, e1 = nullptr;
+    if (prof) {
+        GC_CUDA_TRY(cudaEventCreate(&e0));
+        GC_CUDA_TRY(cudaEventCreate(&e1));
+        GC_CUDA_TRY(cudaEventRecord(e0, g->stream));
+    }
+    int blocks = 0;
+    rc = prof ? launch<true>(g, a, &blocks) : launch<false>(g, a, &blocks);
+    if (rc) return rc;
+    r->launches += 2;  // fill + persistent kernel
+    if (prof) GC_CUDA_TRY(cudaEventRecord(e1, g->stream));
+    unsigned long long h[16];
+    GC_CUDA_TRY(cudaMemcpyAsync(h, s.ctr + kRem, sizeof(h), cudaMemcpyDeviceToHost, g->stream));
+    GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
+    if (h[0] != 0) {
+        set_error("max-min colouring exceeded the round limit");
+        return GC_ERR_TOO_LARGE;
+    }
+    r->rounds = (int64_t)h[kRounds - kRem];
+    r->inner = r->rounds;
+    if (prof) {
+        float ms = 0.f;
+        cudaEventElapsedTime(&ms, e0, e1);
+        cudaEventDestroy(e0);
+        cudaEventDestroy(e1);
+        p.prof->ms[0] += ms;
+        p.prof->launches[0] += 1;
+        p.prof->launch_us.push_back(1e3f * ms);
+        // phase split (globaltimer, block 0): stored in ms[1..3] as fractions
+        const double ns1 = (double)h[kPhaseNs - kRem], ns2 = (double)h[kPhaseNs + 1 - kRem],
+                     ns3 = (double)h[kPhaseNs + 2 - kRem];
+        p.prof->ms[1] += ns1 / 1e6;
+        p.prof->ms[2] += ns2 / 1e6;
+        p.prof->ms[3] += ns3 / 1e6;
+        const int64_t visE = (int64_t)h[kVisE - kRem], visS = (int64_t)h[kVisS - kRem],
+                      visN = (int64_t)h[kVisN - kRem], sumD = (int64_t)h[kSumD - kRem];
+        // algorithmic bytes of the whole persistent kernel: per
+        // evaluated vertex 4 B (D entry, not in round 0) + 16 B row offsets +
+        // 16 B witness state (not in round 0) + 16 B state or 8 B colour/list
+        // write; 4 B per scanned entry; per coloured vertex 4 B list + 16 B
+        // offsets; 4 B per notified entry.
+        const int64_t b = 4 * (sumD - n) + 16 * sumD + 16 * (sumD - n) + 16 * (sumD - n) + 8 * n +
+                          4 * (visE + visS) + 20 * n + 4 * visN;
+        p.prof->bytes[0] += b;
+        p.prof->visits += visE + visS;
+    }
+    return GC_OK;
+}
+
+}  // namespace gc
