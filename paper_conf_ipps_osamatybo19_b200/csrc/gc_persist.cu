@@ -85,6 +85,17 @@ struct Args {
     uint32_t max_rounds;
 };
 
+// Grid-wide phase boundary.  Every phase reads state other SMs wrote in the
+// previous phase (colours, witnesses, queues, long-scan slots are rewritten
+// every round) and L1 is not coherent, so each thread issues a gpu-scope fence
+// after the barrier: it invalidates the SM's L1 (CCTL.IVALL) before the
+// phase's first load.  Without it wake() can read a stale UNC colour and
+// re-enqueue a vertex coloured this round.
+__device__ __forceinline__ void phase_barrier(cg::grid_group &grid) {
+    grid.sync();
+    __threadfence();
+}
+
 __device__ __forceinline__ unsigned long long gtimer() {
     unsigned long long t;
     asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
@@ -307,7 +318,7 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
             for (unsigned long long i = gwarp; i < N; i += nwarps)
                 eval_warp<PROF>(a, cs, Din[i], k, false, nvisE);
         }
-        grid.sync();
+        phase_barrier(grid);
         if (PROF && gtid == 0) {
             unsigned long long t = gtimer();
             tacc[0] += t - t0;
@@ -318,14 +329,14 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
         if (nwq) {
             for (unsigned long long i = gwarp; i < nwq; i += nwarps)
                 eval_warp<PROF>(a, cs, a.WQ[i], k, dense, nvisE);
-            grid.sync();
+            phase_barrier(grid);
         }
         // ------------------------------------------------------------ P2
         const unsigned long long nsq = cs[cSQ];
         if (nsq) {
             for (unsigned long long i = gwarp; i < nsq; i += nwarps)
                 scan_segment<PROF>(a, cs, a.SQ[i], k, dense, nvisS);
-            grid.sync();
+            phase_barrier(grid);
         }
         if (PROF && gtid == 0) {
             unsigned long long t = gtimer();
@@ -372,7 +383,7 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
             a.rstat[4 * k + 3] = (int64_t)nq;
         }
         rem -= ncol;
-        grid.sync();
+        phase_barrier(grid);
         if (PROF && gtid == 0) {
             unsigned long long t = gtimer();
             tacc[2] += t - t0;
