@@ -20,6 +20,8 @@
 // The host launches one kernel per colouring; per-round sizes land in nk[].
 #include <cooperative_groups.h>
 
+#include <cstdio>
+
 #include "gc_event_common.cuh"
 
 namespace cg = cooperative_groups;
@@ -83,7 +85,18 @@ struct Args {
     int64_t n;
     uint32_t key;
     uint32_t max_rounds;
+    unsigned long long nq_cap, sq_cap, ls_cap;  // queue capacities (items)
 };
+
+// Internal-consistency trap: record the first violation (kind, round, vertex)
+// in ctr[kErr..kErr+2] instead of writing out of bounds.
+enum : int { kErr = 56 };
+__device__ __forceinline__ void flag_error(const Args &a, unsigned kind, uint32_t k, uint32_t v) {
+    if (atomicCAS(&a.ctr[kErr], 0ull, (unsigned long long)kind) == 0ull) {
+        a.ctr[kErr + 1] = k;
+        a.ctr[kErr + 2] = v;
+    }
+}
 
 // Grid-wide phase boundary.  Every phase reads state other SMs wrote in the
 // previous phase (colours, witnesses, queues, long-scan slots are rewritten
@@ -119,6 +132,10 @@ __device__ __forceinline__ void enqueue_notify(const Args &a, unsigned long long
         unsigned long long b = 0;
         if (lane_id() == 0) b = atomicAdd(&cs[cNQ], (unsigned long long)nseg);
         b = __shfl_sync(kFull, b, 0);
+        if (b + nseg > a.nq_cap) {
+            if (lane_id() == 0) flag_error(a, 1, 0, uu);
+            continue;
+        }
         for (uint32_t q = lane_id(); q < nseg; q += 32) a.NQ[b + q] = make_uint2(uu, q);
     }
     const unsigned m = __ballot_sync(kFull, colored);
@@ -151,6 +168,15 @@ __device__ __forceinline__ void eval_warp(const Args &a, unsigned long long *cs,
         unsigned long long slot = 0, b = 0;
         if (lane == 0) {
             slot = atomicAdd(&cs[cLS], 1ull);
+            b = atomicAdd(&cs[cSQ], (unsigned long long)nseg);
+            if (slot >= a.ls_cap || b + nseg > a.sq_cap) {
+                flag_error(a, 2, k, v);
+                slot = ~0ull;
+            }
+        }
+        slot = __shfl_sync(kFull, slot, 0);
+        if (slot == ~0ull) return;
+        if (lane == 0) {
             LongScan L;
             L.v = v;
             L.ticket = nseg;
@@ -161,15 +187,16 @@ __device__ __forceinline__ void eval_warp(const Args &a, unsigned long long *cs,
             L.sl = (uint32_t)(r.sl - rs);
             L.base = (uint32_t)(lim - rs);
             a.LS[slot] = L;
-            b = atomicAdd(&cs[cSQ], (unsigned long long)nseg);
         }
-        slot = __shfl_sync(kFull, slot, 0);
         b = __shfl_sync(kFull, b, 0);
         for (uint32_t q = lane; q < nseg; q += 32) a.SQ[b + q] = make_uint2((uint32_t)slot, q);
         return;
     }
     bool colored = false;
-    if (lane == 0) colored = settle(v, rs, r, f, k, a.C, a.W, a.P);
+    if (lane == 0) {
+        if (a.C[v] != GC_UNC) flag_error(a, 3, k, v);
+        colored = settle(v, rs, r, f, k, a.C, a.W, a.P);
+    }
     colored = __shfl_sync(kFull, colored, 0);
     enqueue_notify(a, cs, colored && lane == 0, v, re - rs);
 }
@@ -248,6 +275,7 @@ __device__ __forceinline__ void scan_segment(const Args &a, unsigned long long *
             f.lpos = rs + mL;
             f.lw = a.ci[f.lpos];
         }
+        if (a.C[v] != GC_UNC) flag_error(a, 4, k, v);
         colored = settle(v, rs, r, f, k, a.C, a.W, a.P);
     }
     colored = __shfl_sync(kFull, colored, 0);
@@ -310,7 +338,10 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
                 const bool unresolved =
                     work && lim < re && ((r.need_hi && f.hpos < 0) || (r.need_lo && f.lpos < 0));
                 bool colored = false;
-                if (work && !unresolved) colored = settle(v, rs, r, f, k, a.C, a.W, a.P);
+                if (work && !unresolved) {
+                    if (a.C[v] != GC_UNC) flag_error(a, 5, k, v);
+                    colored = settle(v, rs, r, f, k, a.C, a.W, a.P);
+                }
                 warp_append(unresolved, v, a.WQ, &cs[cWQ]);
                 enqueue_notify(a, cs, colored, v, re - rs);
             }
@@ -435,7 +466,7 @@ int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     int rc = fill_u32(s.C, GC_UNC, n, g->stream);  // Alg.5 L5
     if (rc) return rc;
     GC_CUDA_TRY(cudaMemsetAsync(s.S, 0, sizeof(uint32_t) * (size_t)n, g->stream));
-    GC_CUDA_TRY(cudaMemsetAsync(s.ctr, 0, 56 * sizeof(unsigned long long), g->stream));
+    GC_CUDA_TRY(cudaMemsetAsync(s.ctr, 0, 64 * sizeof(unsigned long long), g->stream));
     const unsigned long long rem = (unsigned long long)n;
     GC_CUDA_TRY(cudaMemcpyAsync(s.ctr + kRem, &rem, sizeof(rem), cudaMemcpyHostToDevice, g->stream));
     const int64_t max_rounds = std::min<int64_t>(p.max_rounds, 0xFFFFFFF0ll);
@@ -462,6 +493,8 @@ int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     a.n = n;
     a.key = p.keys.k[0];
     a.max_rounds = (uint32_t)max_rounds;
+    a.nq_cap = a.sq_cap = (unsigned long long)(n + g->nnz / 128 + 1);
+    a.ls_cap = (unsigned long long)n;
     const bool prof = p.prof && p.prof->on;
     cudaEvent_t e0 = nullptr, e1 = nullptr;
     if (prof) {
@@ -474,9 +507,16 @@ int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     if (rc) return rc;
     r->launches += 2;  // fill + persistent kernel
     if (prof) GC_CUDA_TRY(cudaEventRecord(e1, g->stream));
-    unsigned long long h[16];
+    unsigned long long h[24];
     GC_CUDA_TRY(cudaMemcpyAsync(h, s.ctr + kRem, sizeof(h), cudaMemcpyDeviceToHost, g->stream));
     GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
+    if (h[kErr - kRem] != 0) {
+        char buf[160];
+        snprintf(buf, sizeof(buf), "internal consistency check %llu failed in round %llu (vertex %llu)",
+                 h[kErr - kRem], h[kErr - kRem + 1], h[kErr - kRem + 2]);
+        set_error(buf);
+        return GC_ERR_CUDA;
+    }
     if (h[0] != 0) {
         set_error("max-min colouring exceeded the round limit");
         return GC_ERR_TOO_LARGE;
