@@ -207,12 +207,24 @@ __device__ __forceinline__ void scan_segment(const Args &a, unsigned long long *
                                              uint32_t k, bool dense, uint32_t &nvis) {
     const unsigned lane = lane_id();
     const uint32_t thresh = 2u * k;
+    if (item.x >= __ldcg(&cs[cLS])) {  // trap: segment of a slot not opened this round
+        if (lane == 0) flag_error(a, 10, k, item.x);
+        return;
+    }
     LongScan *L = &a.LS[item.x];
     const uint32_t v = L->v;
     const uint32_t need = L->need;
+    if (v >= (uint32_t)a.n) {
+        if (lane == 0) flag_error(a, 11, k, v);
+        return;
+    }
     const int64_t rs = a.ro[v], re = a.ro[v + 1];
     const int64_t e0 = rs + (int64_t)L->base + (int64_t)item.y * kSeg;
     const int64_t e1 = min(re, e0 + (int64_t)kSeg);
+    if (e0 >= re) {
+        if (lane == 0) flag_error(a, 12, k, v);
+        return;
+    }
     const uint32_t pv = weight_mix(v ^ a.key);
     // skip when every needed side already has a hit before this segment
     const uint32_t curH = *(volatile uint32_t *)&L->minH, curL = *(volatile uint32_t *)&L->minL;
@@ -265,18 +277,21 @@ __device__ __forceinline__ void scan_segment(const Args &a, unsigned long long *
     if (lane == 0) {
         __threadfence();
         const uint32_t mH = atomicAdd(&L->minH, 0u), mL = atomicAdd(&L->minL, 0u);
+        const bool bad = (mH != kNone && mH >= (uint32_t)(re - rs)) ||
+                         (mL != kNone && mL >= (uint32_t)(re - rs));
+        if (bad) flag_error(a, 13 + (mH != kNone && mH >= (uint32_t)(re - rs) ? 0 : 1), k, v);
         const Resume r = resume_of(v, rs, dense, a.W, a.P, a.C, thresh);
         Found f;
-        if (mH != kNone) {
+        if (mH != kNone && !bad) {
             f.hpos = rs + mH;
             f.hw = a.ci[f.hpos];
         }
-        if (mL != kNone) {
+        if (mL != kNone && !bad) {
             f.lpos = rs + mL;
             f.lw = a.ci[f.lpos];
         }
         if (a.C[v] != GC_UNC) flag_error(a, 4, k, v);
-        colored = settle(v, rs, r, f, k, a.C, a.W, a.P);
+        if (!bad) colored = settle(v, rs, r, f, k, a.C, a.W, a.P);
     }
     colored = __shfl_sync(kFull, colored, 0);
     enqueue_notify(a, cs, colored && lane == 0, v, re - rs);
