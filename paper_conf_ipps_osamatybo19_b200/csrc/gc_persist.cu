@@ -90,12 +90,15 @@ struct Args {
 
 // Internal-consistency trap: record the first violation (kind, round, vertex)
 // in ctr[kErr..kErr+2] instead of writing out of bounds.
-enum : int { kErr = 56 };
+// ctr[kErrPar + (k & 1)] marks "a trap fired in round k"; it is read at the
+// top of round k+1, after the barrier, so the exit decision is grid-uniform.
+enum : int { kErr = 56, kErrPar = 59 };
 __device__ __forceinline__ void flag_error(const Args &a, unsigned kind, uint32_t k, uint32_t v) {
     if (atomicCAS(&a.ctr[kErr], 0ull, (unsigned long long)kind) == 0ull) {
         a.ctr[kErr + 1] = k;
         a.ctr[kErr + 2] = v;
     }
+    a.ctr[kErrPar + (k & 1)] = 1;
 }
 
 // Grid-wide phase boundary.  Every phase reads state other SMs wrote in the
@@ -119,7 +122,7 @@ __device__ __forceinline__ unsigned long long gtimer() {
 // (whole warp converged).  Short rows -> NQS (one lane each); long rows ->
 // NQ segments.
 __device__ __forceinline__ void enqueue_notify(const Args &a, unsigned long long *cs, bool colored,
-                                               uint32_t u, int64_t deg) {
+                                               uint32_t u, int64_t deg, uint32_t k) {
     const bool shortrow = colored && deg <= kLaneNotify;
     warp_append(shortrow, u, a.NQS, &cs[cNQS]);
     unsigned lm = __ballot_sync(kFull, colored && !shortrow);
@@ -133,7 +136,7 @@ __device__ __forceinline__ void enqueue_notify(const Args &a, unsigned long long
         if (lane_id() == 0) b = atomicAdd(&cs[cNQ], (unsigned long long)nseg);
         b = __shfl_sync(kFull, b, 0);
         if (b + nseg > a.nq_cap) {
-            if (lane_id() == 0) flag_error(a, 1, 0, uu);
+            if (lane_id() == 0) flag_error(a, 1, k, uu);
             continue;
         }
         for (uint32_t q = lane_id(); q < nseg; q += 32) a.NQ[b + q] = make_uint2(uu, q);
@@ -198,7 +201,7 @@ __device__ __forceinline__ void eval_warp(const Args &a, unsigned long long *cs,
         colored = settle(v, rs, r, f, k, a.C, a.W, a.P);
     }
     colored = __shfl_sync(kFull, colored, 0);
-    enqueue_notify(a, cs, colored && lane == 0, v, re - rs);
+    enqueue_notify(a, cs, colored && lane == 0, v, re - rs, k);
 }
 
 // One kSeg-entry segment of a long scan (whole warp).
@@ -294,7 +297,7 @@ __device__ __forceinline__ void scan_segment(const Args &a, unsigned long long *
         if (!bad) colored = settle(v, rs, r, f, k, a.C, a.W, a.P);
     }
     colored = __shfl_sync(kFull, colored, 0);
-    enqueue_notify(a, cs, colored && lane == 0, v, re - rs);
+    enqueue_notify(a, cs, colored && lane == 0, v, re - rs, k);
 }
 
 template <bool PROF>
@@ -313,6 +316,7 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
         unsigned long long *cn = a.ctr + kSet + 8 * ((k + 1) & 1);
         if (gtid == 0 && (int64_t)k < a.nk_cap) a.nk[k] = (int64_t)rem;
         if (rem == 0 || k >= a.max_rounds) break;  // uniform: rem is computed identically
+        if (k > 0 && __ldcg(&a.ctr[kErrPar + ((k - 1) & 1)]) != 0) break;  // a trap fired
         const bool dense = k == 0;
         const unsigned long long N = dense ? (unsigned long long)a.n : cs[cD];
         if (gtid == 0) {
@@ -358,7 +362,7 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
                     colored = settle(v, rs, r, f, k, a.C, a.W, a.P);
                 }
                 warp_append(unresolved, v, a.WQ, &cs[cWQ]);
-                enqueue_notify(a, cs, colored, v, re - rs);
+                enqueue_notify(a, cs, colored, v, re - rs, k);
             }
         } else {
             for (unsigned long long i = gwarp; i < N; i += nwarps)
@@ -484,7 +488,10 @@ int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     GC_CUDA_TRY(cudaMemsetAsync(s.ctr, 0, 64 * sizeof(unsigned long long), g->stream));
     const unsigned long long rem = (unsigned long long)n;
     GC_CUDA_TRY(cudaMemcpyAsync(s.ctr + kRem, &rem, sizeof(rem), cudaMemcpyHostToDevice, g->stream));
-    const int64_t max_rounds = std::min<int64_t>(p.max_rounds, 0xFFFFFFF0ll);
+    // a round with >= 2 uncoloured vertices colours at least the global max
+    // and min among them, so R <= n/2 + 1
+    const int64_t max_rounds = std::min<int64_t>(std::min<int64_t>(p.max_rounds, 0xFFFFFFF0ll),
+                                                 n / 2 + 2);
     rc = ensure_nk(g, std::min<int64_t>(std::min<int64_t>(n + 2, max_rounds + 2), 1 << 20));
     if (rc) return rc;
     Args a;
