@@ -18,13 +18,11 @@
 // A phase whose queue is empty is skipped (its barrier too): the decision is
 // taken after a barrier from device counters, so it is grid-uniform.
 // The host launches one kernel per colouring; per-round sizes land in nk[].
-#include <cooperative_groups.h>
 
 #include <cstdio>
 
 #include "gc_event_common.cuh"
 
-namespace cg = cooperative_groups;
 
 namespace gc {
 
@@ -101,21 +99,58 @@ __device__ __forceinline__ void flag_error(const Args &a, unsigned kind, uint32_
     a.ctr[kErrPar + (k & 1)] = 1;
 }
 
-// Grid-wide phase boundary.  Every phase reads state other SMs wrote in the
-// previous phase (colours, witnesses, queues, long-scan slots are rewritten
-// every round) and L1 is not coherent, so each thread issues a gpu-scope fence
-// after the barrier: it invalidates the SM's L1 (CCTL.IVALL) before the
-// phase's first load.  Without it wake() can read a stale UNC colour and
-// re-enqueue a vertex coloured this round.
-__device__ __forceinline__ void phase_barrier(cg::grid_group &grid) {
-    grid.sync();
-    __threadfence();
-}
-
 __device__ __forceinline__ unsigned long long gtimer() {
     unsigned long long t;
     asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
     return t;
+}
+
+// Grid-wide phase boundary (the kernel is launched cooperatively, so every
+// block is resident).  Generation barrier on ctr[kBar], ctr[kBar+1]: the last
+// block to arrive resets the count and bumps the generation.  A wait longer
+// than kBarrierTimeoutNs records a trap and makes every block leave the
+// kernel (returns false) instead of hanging the GPU.  Every thread then
+// issues a gpu-scope fence: the next phase reads state other SMs wrote (L1 is
+// not coherent; the fence invalidates it).
+enum : int { kBar = 61, kAbort = 63 };
+constexpr unsigned long long kBarrierTimeoutNs = 4000000000ull;
+
+__device__ __forceinline__ bool phase_barrier(const Args &a, int id, uint32_t k) {
+    __shared__ int ok_sh;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        int ok = 1;
+        volatile unsigned long long *gen = a.ctr + kBar + 1;
+        volatile unsigned long long *abort = a.ctr + kAbort;
+        const unsigned long long g0 = *gen;
+        __threadfence();
+        const unsigned long long arrived = atomicAdd(a.ctr + kBar, 1ull) + 1;
+        if (arrived == gridDim.x) {
+            a.ctr[kBar] = 0;
+            __threadfence();
+            atomicAdd(a.ctr + kBar + 1, 1ull);
+        } else {
+            const unsigned long long t0 = gtimer();
+            while (*gen == g0) {
+                if (*abort) {
+                    ok = 0;
+                    break;
+                }
+                if (gtimer() - t0 > kBarrierTimeoutNs) {
+                    flag_error(a, 100 + id, k, blockIdx.x);
+                    atomicExch(a.ctr + kAbort, 1ull);
+                    ok = 0;
+                    break;
+                }
+                __nanosleep(64);
+            }
+        }
+        __threadfence();
+        ok_sh = ok;
+    }
+    __syncthreads();
+    __threadfence();
+    return ok_sh != 0;
 }
 
 // Enqueue the notification work of lanes whose vertex was just coloured
@@ -302,7 +337,6 @@ __device__ __forceinline__ void scan_segment(const Args &a, unsigned long long *
 
 template <bool PROF>
 __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
-    cg::grid_group grid = cg::this_grid();
     const unsigned lane = lane_id();
     const unsigned long long gtid = (unsigned long long)blockIdx.x * blockDim.x + threadIdx.x;
     const unsigned long long nthreads = (unsigned long long)gridDim.x * blockDim.x;
@@ -368,7 +402,7 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
             for (unsigned long long i = gwarp; i < N; i += nwarps)
                 eval_warp<PROF>(a, cs, Din[i], k, false, nvisE);
         }
-        phase_barrier(grid);
+        if (!phase_barrier(a, 0, k)) return;
         if (PROF && gtid == 0) {
             unsigned long long t = gtimer();
             tacc[0] += t - t0;
@@ -379,14 +413,14 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
         if (nwq) {
             for (unsigned long long i = gwarp; i < nwq; i += nwarps)
                 eval_warp<PROF>(a, cs, a.WQ[i], k, dense, nvisE);
-            phase_barrier(grid);
+            if (!phase_barrier(a, 1, k)) return;
         }
         // ------------------------------------------------------------ P2
         const unsigned long long nsq = cs[cSQ];
         if (nsq) {
             for (unsigned long long i = gwarp; i < nsq; i += nwarps)
                 scan_segment<PROF>(a, cs, a.SQ[i], k, dense, nvisS);
-            phase_barrier(grid);
+            if (!phase_barrier(a, 2, k)) return;
         }
         if (PROF && gtid == 0) {
             unsigned long long t = gtimer();
@@ -433,7 +467,7 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
             a.rstat[4 * k + 3] = (int64_t)nq;
         }
         rem -= ncol;
-        phase_barrier(grid);
+        if (!phase_barrier(a, 3, k)) return;
         if (PROF && gtid == 0) {
             unsigned long long t = gtimer();
             tacc[2] += t - t0;
