@@ -335,6 +335,61 @@ __device__ __forceinline__ void scan_segment(const Args &a, unsigned long long *
     enqueue_notify(a, cs, colored && lane == 0, v, re - rs, k);
 }
 
+// Lane-serial search of a short window [s, lim) (lim - s <= WIN): all column
+// indices first, then all colours, then the in-order first-hit test, so the
+// lane waits for two dependent loads instead of 2 * WIN.
+template <int WIN>
+__device__ __forceinline__ void lane_window(const Args &a, uint32_t thresh, uint32_t pv,
+                                            const Resume &r, int64_t s, int64_t lim, Found &f) {
+    uint32_t u[WIN], c[WIN];
+#pragma unroll
+    for (int q = 0; q < WIN; ++q) u[q] = s + q < lim ? a.ci[s + q] : 0u;
+#pragma unroll
+    for (int q = 0; q < WIN; ++q) c[q] = s + q < lim ? a.C[u[q]] : 0u;
+#pragma unroll
+    for (int q = 0; q < WIN; ++q) {
+        const int64_t e = s + q;
+        if (e < lim && c[q] >= thresh) {
+            const uint32_t pu = weight_mix(u[q] ^ a.key);
+            if (r.need_hi && f.hpos < 0 && e >= r.sh && pu > pv) {
+                f.hpos = e;
+                f.hw = u[q];
+            }
+            if (r.need_lo && f.lpos < 0 && e >= r.sl && pu < pv) {
+                f.lpos = e;
+                f.lw = u[q];
+            }
+        }
+    }
+}
+
+// Wake the neighbours at e0, e0+stride, ... (< re) of vertex u coloured in
+// round k (whole warp converged; u == kNone for idle lanes).  Loads are issued
+// level by level -- all column indices, then all colours, then the witnesses
+// of the uncoloured ones -- so one lane's Q gathers overlap.
+template <int Q>
+__device__ __forceinline__ void notify_entries(const Args &a, uint32_t u, int64_t e0, int64_t re,
+                                               int stride, uint32_t k, uint32_t *Dout,
+                                               unsigned long long *dcount) {
+    uint32_t w[Q], cw[Q];
+    uint2 ww[Q];
+#pragma unroll
+    for (int q = 0; q < Q; ++q) {
+        const int64_t e = e0 + (int64_t)q * stride;
+        w[q] = (u != kNone && e < re) ? a.ci[e] : kNone;
+    }
+#pragma unroll
+    for (int q = 0; q < Q; ++q) cw[q] = w[q] != kNone ? a.C[w[q]] : 0u;
+#pragma unroll
+    for (int q = 0; q < Q; ++q) ww[q] = cw[q] == GC_UNC ? a.W[w[q]] : make_uint2(kNone, kNone);
+#pragma unroll
+    for (int q = 0; q < Q; ++q) {
+        bool wk = cw[q] == GC_UNC && (ww[q].x == u || ww[q].y == u);
+        if (wk) wk = atomicMax(&a.S[w[q]], k + 1u) < k + 1u;
+        warp_append(wk, w[q], Dout, dcount);
+    }
+}
+
 template <bool PROF>
 __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
     const unsigned lane = lane_id();
@@ -383,11 +438,8 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
                 if (r.need_lo && r.sl < s) s = r.sl;
                 const int64_t lim = min(re, s + (int64_t)kLaneWin);
                 Found f;
-                uint32_t vis = 0;
-                if (work)
-                    lane_search(a.ci, a.C, thresh, a.key, weight_mix(v ^ a.key), r.need_hi,
-                                r.need_lo, r.sh, r.sl, lim, f, vis);
-                if (PROF) nvisE += vis;
+                if (work) lane_window<kLaneWin>(a, thresh, weight_mix(v ^ a.key), r, s, lim, f);
+                if (PROF && work) nvisE += (uint32_t)(lim - s);
                 const bool unresolved =
                     work && lim < re && ((r.need_hi && f.hpos < 0) || (r.need_lo && f.lpos < 0));
                 bool colored = false;
@@ -431,34 +483,26 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
         const unsigned long long ncol = cs[cI];
         const unsigned long long nqs = cs[cNQS], nq = cs[cNQ];
         unsigned long long *dcount = &cn[cD];
-        for (unsigned long long base = gwarp * 32; base < nqs; base += nthreads) {
-            const unsigned long long idx = base + lane;
+        // short rows: 4 rows per warp, 8 lanes per row, 4 entries per lane
+        for (unsigned long long base = gwarp * 4; base < nqs; base += nwarps * 4) {
+            const unsigned long long idx = base + (lane >> 3);
+            uint32_t u = kNone;
+            int64_t rs = 0, re = 0;
             if (idx < nqs) {
-                const uint32_t u = a.NQS[idx];
-                const int64_t rs = a.ro[u], re = a.ro[u + 1];
-                for (int64_t e = rs; e < re; ++e) {
-                    const uint32_t w = a.ci[e];
-                    if (wake(w, u, k, a.C, a.W, a.S)) Dout[atomicAdd(dcount, 1ull)] = w;
-                }
-                if (PROF) nvisN += (uint32_t)(re - rs);
+                u = a.NQS[idx];
+                rs = a.ro[u];
+                re = a.ro[u + 1];
             }
+            notify_entries<4>(a, u, rs + (lane & 7), re, 8, k, Dout, dcount);
+            if (PROF && (lane & 7) == 0) nvisN += (uint32_t)(re - rs);
         }
+        // long rows: one kNotifySeg-entry segment per warp
         for (unsigned long long it = gwarp; it < nq; it += nwarps) {
             const uint2 item = a.NQ[it];
             const uint32_t u = item.x;
             const int64_t rs = a.ro[u] + (int64_t)item.y * kNotifySeg;
             const int64_t re = min(a.ro[u + 1], rs + (int64_t)kNotifySeg);
-            uint32_t w[kNotifySeg / 32];
-#pragma unroll
-            for (int q = 0; q < kNotifySeg / 32; ++q) {
-                const int64_t e = rs + q * 32 + lane;
-                w[q] = e < re ? a.ci[e] : kNone;
-            }
-#pragma unroll
-            for (int q = 0; q < kNotifySeg / 32; ++q) {
-                const bool wk = w[q] != kNone && wake(w[q], u, k, a.C, a.W, a.S);
-                warp_append(wk, w[q], Dout, dcount);
-            }
+            notify_entries<kNotifySeg / 32>(a, u, rs + lane, re, 32, k, Dout, dcount);
             if (PROF && lane == 0) nvisN += (uint32_t)(re - rs);
         }
         if (PROF && gtid == 0 && (int64_t)k < a.nk_cap) {
