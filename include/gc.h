@@ -204,6 +204,15 @@ int gc_create_csr_dist(int64_t n_global, int64_t v_begin, int64_t v_end,
 /* Fill 128 bytes with a fresh NCCL unique id (call on rank 0 only). */
 int gc_nccl_unique_id(void *out128);
 
+/* The partitioned algorithm of gc_create_csr_dist run on ONE GPU: the graph
+ * (same arguments as gc_create_csr) is split into `parts` equal vertex ranges,
+ * each with its own colour replica, exchanged every round by device copies
+ * instead of NCCL.  gc_color on the handle returns exactly the single-GPU
+ * colouring; this is how the partition / exchange logic is tested on one GPU. */
+int gc_create_csr_loopback(int64_t n, int64_t nnz, const int64_t *row_offsets,
+                           const uint32_t *col_indices, int parts, uint32_t flags,
+                           gc_graph **out);
+
 #ifdef __cplusplus
 }
 #endif

@@ -40,7 +40,7 @@ MODE_AUTO, MODE_SWEEP, MODE_EVENT, MODE_EVENT_MULTI = 0, 1, 2, 3
 
 EXPORTS = ["gc_create_csr", "gc_color", "gc_color_ex", "gc_set_stream", "gc_destroy",
            "gc_last_error", "gc_priorities", "gc_count_colors", "gc_version",
-           "gc_create_csr_dist", "gc_nccl_unique_id"]
+           "gc_create_csr_dist", "gc_nccl_unique_id", "gc_create_csr_loopback"]
 
 
 class GCError(RuntimeError):
@@ -98,6 +98,8 @@ def lib():
                                          u32, ctypes.POINTER(P)]
         L.gc_create_csr_dist.restype = ctypes.c_int
         L.gc_nccl_unique_id.argtypes, L.gc_nccl_unique_id.restype = [P], ctypes.c_int
+        L.gc_create_csr_loopback.argtypes = [i64, i64, P, P, ctypes.c_int, u32, ctypes.POINTER(P)]
+        L.gc_create_csr_loopback.restype = ctypes.c_int
         _lib = L
     return _lib
 
@@ -225,6 +227,38 @@ class Graph:
 
     def __exit__(self, *a):
         self.close()
+
+
+def loopback_graph(n: int, row_offsets, col_indices, parts: int, flags: int = 0) -> Graph:
+    """The partitioned (multi-GPU) algorithm with `parts` partitions on this GPU."""
+    h = ctypes.c_void_p()
+    nnz = int(col_indices.numel() if hasattr(col_indices, "numel") else col_indices.size)
+    _check(lib().gc_create_csr_loopback(n, nnz, _ptr(row_offsets, ("int64",)),
+                                        _ptr(col_indices, ("int32", "uint32")), parts, flags,
+                                        ctypes.byref(h)))
+    return Graph._from_handle(h, n, nnz)
+
+
+def nccl_unique_id() -> bytes:
+    buf = ctypes.create_string_buffer(128)
+    _check(lib().gc_nccl_unique_id(buf))
+    return buf.raw
+
+
+def dist_graph(n_global: int, v_begin: int, v_end: int, row_offsets_local, col_indices_global,
+               unique_id: bytes, rank: int, world: int, flags: int = 0) -> Graph:
+    """A rank's share of a 1D-partitioned graph (collective over `world` ranks)."""
+    h = ctypes.c_void_p()
+    nnz = int(col_indices_global.numel())
+    uid = ctypes.create_string_buffer(bytes(unique_id), 128)
+    _check(lib().gc_create_csr_dist(n_global, v_begin, v_end, nnz,
+                                    _ptr(row_offsets_local, ("int64",)),
+                                    _ptr(col_indices_global, ("int32", "uint32")), uid, rank,
+                                    world, flags, ctypes.byref(h)))
+    g = Graph._from_handle(h, n_global, nnz,
+                           keep=(row_offsets_local, col_indices_global) if flags & BORROW_DEVICE
+                           else None)
+    return g
 
 
 def color(n, row_offsets, col_indices, seed=1, variant=MAXMIN, out=None, **kw):

@@ -325,9 +325,9 @@ const char *gc_version(void) {
     return buf;
 }
 
-static int create_common(int64_t n, int64_t nnz, const int64_t *row_offsets,
-                         const uint32_t *col_indices, uint32_t flags, gc_graph **out,
-                         int64_t v_begin, int64_t n_global) {
+int gc_create_csr_internal(int64_t n, int64_t nnz, const int64_t *row_offsets,
+                           const uint32_t *col_indices, uint32_t flags, gc_graph **out,
+                           int64_t v_begin, int64_t n_global) {
     if (!out) {
         set_error("gc_create_csr: out is NULL");
         return GC_ERR_INVALID_ARG;
@@ -423,7 +423,7 @@ static int create_common(int64_t n, int64_t nnz, const int64_t *row_offsets,
 
 int gc_create_csr(int64_t n, int64_t nnz, const int64_t *row_offsets, const uint32_t *col_indices,
                   uint32_t flags, gc_graph **out) {
-    return create_common(n, nnz, row_offsets, col_indices, flags, out, 0, n);
+    return gc_create_csr_internal(n, nnz, row_offsets, col_indices, flags, out, 0, n);
 }
 
 int gc_set_stream(gc_graph *g, void *cuda_stream) {

@@ -132,6 +132,30 @@ struct RunResult {
     int64_t launches = 0;
 };
 
+// One sweep round over a vertex range [v0, v0 + n_loc) (single GPU: v0 = 0).
+// C is indexed by global vertex id; rows by (v - v0).
+constexpr int kColoredCtr = 16;  // ctr slot counting `colored` pairs
+struct SweepArgs {
+    const int64_t *ro;
+    const uint32_t *ci;
+    uint32_t *C;
+    const uint32_t *Fin;
+    uint32_t *Fout;
+    uint32_t *hub;
+    unsigned long long *ctr;
+    int64_t *nk;
+    int64_t nk_cap;
+    uint32_t k;
+    int H;
+    Keys keys;
+    int dense;
+    int64_t n_loc;
+    uint32_t v0;
+    uint32_t thread_max, hub_min;
+    uint2 *colored;  // optional: (v, colour) of the vertices coloured this round
+};
+int sweep_round(const SweepArgs &a, cudaStream_t st, int blocks_sweep, int blocks_hub);
+
 int ensure_scratch(gc_graph *g, bool need_event, bool need_luby);
 int run_sweep_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int run_event_maxmin(gc_graph *g, const RunParams &p, RunResult *r);

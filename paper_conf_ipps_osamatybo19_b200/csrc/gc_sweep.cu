@@ -93,16 +93,23 @@ __device__ __forceinline__ void warp_append(bool pred, uint32_t v, uint32_t *lis
 }
 
 template <int HT, bool PROF>
-__global__ void __launch_bounds__(kBlock) k_sweep(
-    const int64_t *__restrict__ ro, const uint32_t *__restrict__ ci, uint32_t *C,
-    const uint32_t *__restrict__ Fin, uint32_t *__restrict__ Fout, uint32_t *__restrict__ hub,
-    unsigned long long *ctr, int64_t *nk, int64_t nk_cap, uint32_t k, int H, Keys keys,
-    int dense, int64_t n, uint32_t thread_max, uint32_t hub_min) {
+__global__ void __launch_bounds__(kBlock) k_sweep(SweepArgs a) {
+    const int64_t *__restrict__ ro = a.ro;
+    const uint32_t *__restrict__ ci = a.ci;
+    uint32_t *C = a.C;
+    const uint32_t *__restrict__ Fin = a.Fin;
+    uint32_t *__restrict__ Fout = a.Fout;
+    uint32_t *__restrict__ hub = a.hub;
+    unsigned long long *ctr = a.ctr;
+    const uint32_t k = a.k, thread_max = a.thread_max, hub_min = a.hub_min, v0 = a.v0;
+    const int H = a.H, dense = a.dense;
+    const Keys &keys = a.keys;
+    const int64_t n = a.n_loc;
     const unsigned long long N = dense ? (unsigned long long)n : ctr[k % 3];
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         ctr[(k + 2) % 3] = 0;
         ctr[3 + (k + 1) % 3] = 0;
-        if ((int64_t)k < nk_cap) nk[k] = (int64_t)N;
+        if ((int64_t)k < a.nk_cap) a.nk[k] = (int64_t)N;
     }
     const int nh = HT > 0 ? HT : H;
     const uint32_t full = (nh >= 32) ? kFull : ((1u << nh) - 1u);
@@ -116,9 +123,9 @@ __global__ void __launch_bounds__(kBlock) k_sweep(
         uint32_t v = 0;
         int64_t rs = 0, re = 0;
         if (valid) {
-            v = dense ? (uint32_t)idx : Fin[idx];
-            rs = ro[v];
-            re = ro[v + 1];
+            v = dense ? v0 + (uint32_t)idx : Fin[idx];
+            rs = ro[v - v0];
+            re = ro[v - v0 + 1];
         }
         const int64_t deg = re - rs;
         const bool small = valid && deg <= (int64_t)thread_max;
@@ -175,6 +182,17 @@ __global__ void __launch_bounds__(kBlock) k_sweep(
             if (col != GC_UNC) C[v] = col;  // atomic-free commit (single writer)
         }
         warp_append(handled && col == GC_UNC, v, Fout, &ctr[(k + 1) % 3]);
+        if (a.colored) {  // distributed: publish (v, colour) of this round
+            const bool c = handled && col != GC_UNC;
+            const unsigned m = __ballot_sync(kFull, c);
+            if (m) {
+                const unsigned leader = __ffs(m) - 1;
+                unsigned long long b = 0;
+                if (lane == leader) b = atomicAdd(&ctr[kColoredCtr], (unsigned long long)__popc(m));
+                b = __shfl_sync(kFull, b, leader);
+                if (c) a.colored[b + __popc(m & ((1u << lane) - 1u))] = make_uint2(v, col);
+            }
+        }
         if (PROF) {
             unsigned tot = __reduce_add_sync(kFull, nvis);
             if (lane == 0 && tot) atomicAdd(&ctr[20], (unsigned long long)tot);
@@ -184,12 +202,16 @@ __global__ void __launch_bounds__(kBlock) k_sweep(
 
 // CTA-per-hub scan of round k.  Persistent over the hub list.
 template <int HT, bool PROF>
-__global__ void __launch_bounds__(512) k_hub(const int64_t *__restrict__ ro,
-                                             const uint32_t *__restrict__ ci, uint32_t *C,
-                                             const uint32_t *__restrict__ hub,
-                                             uint32_t *__restrict__ Fout,
-                                             unsigned long long *ctr, uint32_t k, int H,
-                                             Keys keys) {
+__global__ void __launch_bounds__(512) k_hub(SweepArgs a) {
+    const int64_t *__restrict__ ro = a.ro;
+    const uint32_t *__restrict__ ci = a.ci;
+    uint32_t *C = a.C;
+    const uint32_t *__restrict__ hub = a.hub;
+    uint32_t *__restrict__ Fout = a.Fout;
+    unsigned long long *ctr = a.ctr;
+    const uint32_t k = a.k, v0 = a.v0;
+    const int H = a.H;
+    const Keys &keys = a.keys;
     const unsigned long long nhub = ctr[3 + k % 3];
     const int nh = HT > 0 ? HT : H;
     const uint32_t full = (nh >= 32) ? kFull : ((1u << nh) - 1u);
@@ -197,7 +219,7 @@ __global__ void __launch_bounds__(512) k_hub(const int64_t *__restrict__ ro,
     __shared__ uint32_t sh_hi, sh_lo;
     for (unsigned long long i = blockIdx.x; i < nhub; i += gridDim.x) {
         const uint32_t v = hub[i];
-        const int64_t rs = ro[v], re = ro[v + 1];
+        const int64_t rs = ro[v - v0], re = ro[v - v0 + 1];
         uint32_t pv[HT > 0 ? HT : GC_MAX_HASHES];
         own_weights<HT>(v, keys, nh, pv);
         if (threadIdx.x == 0) {
@@ -246,6 +268,7 @@ __global__ void __launch_bounds__(512) k_hub(const int64_t *__restrict__ ro,
             uint32_t col = decide(H_all, L_all, full, k, nh);
             if (col != GC_UNC) {
                 C[v] = col;
+                if (a.colored) a.colored[atomicAdd(&ctr[kColoredCtr], 1ull)] = make_uint2(v, col);
             } else {
                 unsigned long long pos = atomicAdd(&ctr[(k + 1) % 3], 1ull);
                 Fout[pos] = v;
@@ -262,22 +285,42 @@ __global__ void k_fill_u32(uint32_t *p, uint32_t val, int64_t n) {
 }
 
 template <int HT, bool PROF>
+int launch_round_args(const SweepArgs &a, cudaStream_t st, int blocks_sweep, int blocks_hub,
+                      EventTimer *tm) {
+    int rc = 0;
+    if (PROF && (rc = tm->begin(st, 0))) return rc;
+    k_sweep<HT, PROF><<<blocks_sweep, kBlock, 0, st>>>(a);
+    if (PROF && (rc = tm->end(st))) return rc;
+    if (PROF && (rc = tm->begin(st, 1))) return rc;
+    k_hub<HT, PROF><<<blocks_hub, 512, 0, st>>>(a);
+    if (PROF && (rc = tm->end(st))) return rc;
+    return GC_OK;
+}
+
+template <int HT, bool PROF>
 int launch_round(gc_graph *g, const RunParams &p, uint32_t k, int blocks_sweep, int blocks_hub,
                  EventTimer *tm) {
     Scratch &s = g->s;
-    const uint32_t *Fin = s.F[k & 1];
-    uint32_t *Fout = s.F[(k + 1) & 1];
-    int rc = 0;
-    if (PROF && (rc = tm->begin(g->stream, 0))) return rc;
-    k_sweep<HT, PROF><<<blocks_sweep, kBlock, 0, g->stream>>>(
-        g->ro, g->ci, s.C, Fin, Fout, s.hub, s.ctr, s.nk, s.nk_cap, k, p.H, p.keys, k == 0 ? 1 : 0,
-        g->n, (uint32_t)p.thread_deg_max, (uint32_t)p.hub_deg_min);
-    if (PROF && (rc = tm->end(g->stream))) return rc;
-    if (PROF && (rc = tm->begin(g->stream, 1))) return rc;
-    k_hub<HT, PROF><<<blocks_hub, 512, 0, g->stream>>>(g->ro, g->ci, s.C, s.hub, Fout, s.ctr, k,
-                                                       p.H, p.keys);
-    if (PROF && (rc = tm->end(g->stream))) return rc;
-    return GC_OK;
+    SweepArgs a;
+    a.ro = g->ro;
+    a.ci = g->ci;
+    a.C = s.C;
+    a.Fin = s.F[k & 1];
+    a.Fout = s.F[(k + 1) & 1];
+    a.hub = s.hub;
+    a.ctr = s.ctr;
+    a.nk = s.nk;
+    a.nk_cap = s.nk_cap;
+    a.k = k;
+    a.H = p.H;
+    a.keys = p.keys;
+    a.dense = k == 0 ? 1 : 0;
+    a.n_loc = g->n;
+    a.v0 = 0;
+    a.thread_max = (uint32_t)p.thread_deg_max;
+    a.hub_min = (uint32_t)p.hub_deg_min;
+    a.colored = nullptr;
+    return launch_round_args<HT, PROF>(a, g->stream, blocks_sweep, blocks_hub, tm);
 }
 
 }  // namespace
@@ -316,6 +359,15 @@ int EventTimer::drain(Profile *p) {
         p->launch_us.push_back(1e3f * ms);
     }
     used = 0;
+    return GC_OK;
+}
+
+int sweep_round(const SweepArgs &a, cudaStream_t st, int blocks_sweep, int blocks_hub) {
+    EventTimer tm;
+    int rc = a.H == 1 ? launch_round_args<1, false>(a, st, blocks_sweep, blocks_hub, &tm)
+                      : launch_round_args<0, false>(a, st, blocks_sweep, blocks_hub, &tm);
+    if (rc) return rc;
+    GC_CUDA_TRY(cudaGetLastError());
     return GC_OK;
 }
 

@@ -262,3 +262,23 @@ def test_cfg4_rmat_s24_certificate():
     assert O.cert_maxmin(gh, 1, 1, C) == 0
     assert O.check_proper(gh, C) == 0
     assert k == O.count_colors(C) and k in (2 * st.rounds - 1, 2 * st.rounds)
+
+
+# ------------------------------------------------- partitioned (row e)
+@pytest.mark.parametrize("parts", [1, 2, 3, 4, 8])
+def test_loopback_partitions(parts):
+    """The multi-GPU algorithm (per-partition replicas + per-round exchange of
+    coloured pairs) with `parts` partitions on one GPU equals the oracle."""
+    for g, vname, H in ((G.rmat(14, 16, seed=5), "maxmin", 1),
+                        (G.erdos_renyi(50000, 400000, seed=6), "maxmin", 1),
+                        (G.rmat(13, 16, seed=7), "multihash", 3),
+                        (G.csr_from_lists(5, [(0, 1), (1, 2)]), "maxmin", 1)):
+        ref, R, nk = O.color_maxmin(g, 9, H, with_stats=True)
+        with gcb.loopback_graph(g.n, g.row_offsets, g.col_indices, parts) as h:
+            out = torch.empty(g.n, dtype=torch.int32)
+            _, k, st = h.color(9, variant_of(vname, H), out, stats=True, frontier_cap=8192)
+            assert (out.numpy().view(np.uint32) == ref).all(), (parts, g.name)
+            assert st.rounds == R and st.frontier_sizes == nk and k == O.count_colors(ref)
+            outc = torch.empty(g.n, dtype=torch.int32)
+            h.color(9, variant_of(vname, H), outc, flags=gcb.COMPACT)
+            assert (outc.numpy().view(np.uint32) == O.compact_colors(ref)).all()
