@@ -41,20 +41,54 @@ __global__ void k_validate(const int64_t *__restrict__ ro, const uint32_t *__res
                            int64_t n, int64_t nnz, int64_t n_global, int64_t v_begin,
                            unsigned long long *err) {
     // err[0]: non-monotone / out-of-range offsets; err[1]: col >= n; err[2]: self-loop;
-    // err[3]: max degree
-    for (int64_t v = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; v < n;
-         v += (int64_t)gridDim.x * blockDim.x) {
-        int64_t a = ro[v], b = ro[v + 1];
-        if (a > b || a < 0 || b > nnz) {
-            atomicAdd(&err[0], 1ull);
-            continue;
+    // err[3]: max degree.  Rows of <= 32 entries are checked by one lane, longer
+    // rows by the whole warp (coalesced); counts are warp-aggregated.
+    const unsigned lane = threadIdx.x & 31u;
+    unsigned long long bad_off = 0, bad_col = 0, loops = 0, maxdeg = 0;
+    const int64_t stride = (int64_t)gridDim.x * blockDim.x;
+    for (int64_t base = (int64_t)blockIdx.x * blockDim.x + (threadIdx.x & ~31u); base < n;
+         base += stride) {
+        const int64_t v = base + lane;
+        int64_t a0 = 0, b0 = 0;
+        bool ok = false;
+        if (v < n) {
+            a0 = ro[v];
+            b0 = ro[v + 1];
+            ok = a0 <= b0 && a0 >= 0 && b0 <= nnz;
+            if (!ok) ++bad_off;
+            else maxdeg = max(maxdeg, (unsigned long long)(b0 - a0));
         }
-        atomicMax(&err[3], (unsigned long long)(b - a));
-        for (int64_t e = a; e < b; ++e) {
-            uint32_t u = ci[e];
-            if ((int64_t)u >= n_global) atomicAdd(&err[1], 1ull);
-            else if ((int64_t)u == v + v_begin) atomicAdd(&err[2], 1ull);
+        const bool shortrow = ok && b0 - a0 <= 32;
+        if (shortrow)
+            for (int64_t e = a0; e < b0; ++e) {
+                const uint32_t u = ci[e];
+                if ((int64_t)u >= n_global) ++bad_col;
+                else if ((int64_t)u == v + v_begin) ++loops;
+            }
+        unsigned lm = __ballot_sync(0xFFFFFFFFu, ok && !shortrow);
+        while (lm) {
+            const int src = __ffs(lm) - 1;
+            lm &= lm - 1;
+            const int64_t ws = __shfl_sync(0xFFFFFFFFu, a0, src);
+            const int64_t we = __shfl_sync(0xFFFFFFFFu, b0, src);
+            const int64_t wv = __shfl_sync(0xFFFFFFFFu, v, src);
+            for (int64_t e = ws + lane; e < we; e += 32) {
+                const uint32_t u = ci[e];
+                if ((int64_t)u >= n_global) ++bad_col;
+                else if ((int64_t)u == wv + v_begin) ++loops;
+            }
         }
+    }
+    bad_off = __reduce_add_sync(0xFFFFFFFFu, (unsigned)bad_off);
+    bad_col = __reduce_add_sync(0xFFFFFFFFu, (unsigned)min(bad_col, 1ull << 20));
+    loops = __reduce_add_sync(0xFFFFFFFFu, (unsigned)min(loops, 1ull << 20));
+    const unsigned md_hi = __reduce_max_sync(0xFFFFFFFFu, (unsigned)(maxdeg >> 32));
+    const unsigned md_lo = __reduce_max_sync(0xFFFFFFFFu, (unsigned)((maxdeg >> 32) == md_hi ? maxdeg : 0));
+    if (lane == 0) {
+        if (bad_off) atomicAdd(&err[0], bad_off);
+        if (bad_col) atomicAdd(&err[1], bad_col);
+        if (loops) atomicAdd(&err[2], loops);
+        atomicMax(&err[3], ((unsigned long long)md_hi << 32) | md_lo);
     }
 }
 
@@ -301,6 +335,8 @@ static void free_scratch(Scratch &s) {
     cudaFree(s.Q2);
     cudaFree(s.Q3);
     cudaFree(s.LS);
+    cudaFree(s.Qd[0]);
+    cudaFree(s.Qd[1]);
     cudaFree(s.ctr);
     cudaFree(s.nk);
     cudaFree(s.rstat);

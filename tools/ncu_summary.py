@@ -8,10 +8,18 @@
 `full`: the key metrics of a `--set full` capture (DRAM bytes, throughput,
 occupancy, registers, stall reasons)."""
 import csv
+import re
 import io
 import subprocess
 import sys
 from collections import defaultdict
+
+
+def kname(full):
+    """'void gc::<unnamed>::k_sweep<1, false>(gc::SweepArgs)' -> 'k_sweep<1, false>'."""
+    head = full.split("(")[0]
+    m = re.search(r"(\w+)(<[^<>]*>)?\s*$", head)
+    return (m.group(1) + (m.group(2) or "")) if m else head
 
 
 def launches(path):
@@ -28,10 +36,10 @@ def launches(path):
         v = float(r[vi].replace(",", ""))
         unit = r[ui] if ui is not None else "ns"
         v *= {"ns": 1e-3, "usecond": 1.0, "us": 1.0, "msecond": 1e3, "ms": 1e3, "nsecond": 1e-3}.get(unit, 1e-3)
-        name = r[ki].split("(")[0].split("<")[0].replace("void ", "").strip()
+        name = kname(r[ki])
         tot[name] += v
         cnt[name] += 1
-    ours = {k: v for k, v in tot.items() if any(s in k for s in ("gc::", "k_"))}
+    ours = {k: v for k, v in tot.items() if k.startswith("k_")}
     allsum = sum(tot.values())
     oursum = sum(ours.values())
     print(f"source: `{path}` (ncu --metrics gpu__time_duration.sum --clock-control none)\n")
@@ -65,7 +73,7 @@ def full(path):
     print(f"source: `{path}` (ncu --set full --clock-control none --import-source on)\n")
     for r in rows[2:]:
         name = r[hdr.index("Kernel Name")] if "Kernel Name" in hdr else "?"
-        print(f"### `{name.split('(')[0]}`\n")
+        print(f"### `{kname(name)}`\n")
         print("| metric | value | unit |")
         print("|---|---:|---|")
         for k in KEYS:
