@@ -337,6 +337,7 @@ static void free_scratch(Scratch &s) {
     cudaFree(s.LS);
     cudaFree(s.Qd[0]);
     cudaFree(s.Qd[1]);
+    cudaFree(s.qctl);
     cudaFree(s.ctr);
     cudaFree(s.nk);
     cudaFree(s.rstat);

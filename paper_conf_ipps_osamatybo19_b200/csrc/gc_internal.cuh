@@ -51,6 +51,7 @@ struct Scratch {
     void *LS = nullptr;           // persistent event mode: long-scan slots (32 B each)
     void *Qd[2] = {nullptr, nullptr};  // persistent event mode: per-round work queues
     size_t qd_cap = 0;
+    unsigned long long *qctl = nullptr;  // persistent event mode: queue counters
     uint32_t *S = nullptr;        // Luby inner-loop state / event stamps
     uint32_t *W = nullptr;        // event mode: witness pairs (2 per vertex)
     uint32_t *P = nullptr;        // event mode: resume cursors (2 per vertex)

@@ -48,6 +48,7 @@ constexpr int kWarpWin = 256;    // entries a warp scans before splitting
 constexpr int kSeg = 256;        // entries per long-scan segment (8 per lane)
 constexpr int kNotifySeg = 128;  // entries per notify segment (4 per lane)
 constexpr int kLaneNotify = 32;  // rows up to this length are one notify item
+constexpr unsigned long long kDynWarps = 2048;  // warps that serve the dynamic queue
 
 // work items: {a, (type << 28) | b}; type 0 marks an empty slot
 enum : uint32_t { T_NOTIFY = 1u, T_EVAL = 2u, T_SCAN = 3u };
@@ -95,6 +96,7 @@ struct Args {
     uint32_t *B0;    // vertices left blocked by round 0 (round 1 re-checks them)
     LongScan *LS;
     uint2 *Q[2];     // work queues by round parity
+    unsigned long long *qc;  // queue counters: set s, counter c at qc[(8 s + c) * 16]
     unsigned long long *ctr;
     int64_t *nk;
     int64_t *rstat;
@@ -104,6 +106,12 @@ struct Args {
     uint32_t max_rounds;
     unsigned long long q_cap, sq_cap, ls_cap;
 };
+
+// Queue counters live on separate 128-byte lines: idle warps poll qDone/qTail
+// while busy warps update them, and a shared line would serialise both.
+__device__ __forceinline__ unsigned long long *QC(const Args &a, int set, int c) {
+    return a.qc + (8 * set + c) * 16;
+}
 
 __device__ __forceinline__ unsigned long long gtimer() {
     unsigned long long t;
@@ -150,7 +158,7 @@ __device__ __forceinline__ bool grid_barrier(const Args &a, int id, uint32_t k, 
         if (arrived == gridDim.x) {
             a.ctr[kBar] = 0;
             if (reset_set >= 0)
-                for (int i = 0; i < 8; ++i) a.ctr[kQ + 8 * reset_set + i] = 0;
+                for (int i = 0; i < 8; ++i) *QC(a, reset_set, i) = 0;
             __threadfence();
             atomicAdd(a.ctr + kBar + 1, 1ull);
         } else {
@@ -196,7 +204,7 @@ __device__ __forceinline__ void push_items(const Args &a, int q, uint32_t cnt, u
                                            Make make) {
     if (cnt == 0) return;
     unsigned long long b = 0;
-    if (lane_id() == 0) b = atomicAdd(&a.ctr[kQ + 8 * q + qTail], (unsigned long long)cnt);
+    if (lane_id() == 0) b = atomicAdd(QC(a, q, qTail), (unsigned long long)cnt);
     b = __shfl_sync(kFull, b, 0);
     for (uint32_t i = lane_id(); i < cnt; i += 32) put_item(a, q, b + i, make(i), k);
 }
@@ -222,7 +230,7 @@ __device__ __forceinline__ void colored_notify(const Args &a, bool colored, uint
         unsigned long long b = 0;
         const unsigned leader = __ffs(sm) - 1;
         if (lane_id() == leader)
-            b = atomicAdd(&a.ctr[kQ + 8 * q + qTail], (unsigned long long)__popc(sm));
+            b = atomicAdd(QC(a, q, qTail), (unsigned long long)__popc(sm));
         b = __shfl_sync(kFull, b, leader);
         if (shortrow)
             put_item(a, q, b + __popc(sm & ((1u << lane_id()) - 1u)),
@@ -291,7 +299,7 @@ __device__ __forceinline__ void eval_warp(const Args &a, uint32_t v, uint32_t k,
     const bool miss_lo = r.need_lo && f.lpos < 0;
     if (lim < re && (miss_hi || miss_lo)) {
         const uint32_t nseg = (uint32_t)((re - lim + kSeg - 1) / kSeg);
-        unsigned long long *lsc = stat ? &a.ctr[r0LS + 3 * k] : &a.ctr[kQ + 8 * (k & 1) + qLS];
+        unsigned long long *lsc = stat ? &a.ctr[r0LS + 3 * k] : QC(a, k & 1, qLS);
         unsigned long long slot = 0;
         if (lane == 0) {
             slot = atomicAdd(lsc, 1ull);
@@ -346,15 +354,18 @@ __device__ __forceinline__ void scan_segment(const Args &a, uint32_t slot, uint3
     const bool dense = k == 0;
     const unsigned lane = lane_id();
     const uint32_t thresh = 2u * k;
+    // the slot was written by another SM in this phase: bypass L1 (a 128-byte
+    // line holds four slots, so it may be cached from a neighbouring slot)
     LongScan *L = &a.LS[slot];
-    const uint32_t v = L->v;
-    const uint32_t need = L->need;
+    const uint32_t v = __ldcg(&L->v);
+    const uint32_t need = __ldcg(&L->need);
+    const uint32_t Lbase = __ldcg(&L->base), Lsh = __ldcg(&L->sh), Lsl = __ldcg(&L->sl);
     if (v >= (uint32_t)a.n) {
         if (lane == 0) flag_error(a, 11, k, v);
         return;
     }
     const int64_t rs = a.ro[v], re = a.ro[v + 1];
-    const int64_t e0 = rs + (int64_t)L->base + (int64_t)seg * kSeg;
+    const int64_t e0 = rs + (int64_t)Lbase + (int64_t)seg * kSeg;
     const int64_t e1 = min(re, e0 + (int64_t)kSeg);
     if (e0 >= re) {
         if (lane == 0) flag_error(a, 12, k, v);
@@ -385,8 +396,8 @@ __device__ __forceinline__ void scan_segment(const Args &a, uint32_t slot, uint3
             if (e < e1 && c[q] >= thresh) {
                 const uint32_t pu = weight_mix(u[q] ^ a.key);
                 const uint32_t rel = (uint32_t)(e - rs);
-                if (want_hi && rel >= L->sh && pu > pv) rh = min(rh, rel);
-                if (want_lo && rel >= L->sl && pu < pv) rl = min(rl, rel);
+                if (want_hi && rel >= Lsh && pu > pv) rh = min(rh, rel);
+                if (want_lo && rel >= Lsl && pu < pv) rl = min(rl, rel);
             }
         }
         if (PROF) {
@@ -457,8 +468,8 @@ __device__ __forceinline__ void notify_entries(const Args &a, uint32_t u, int64_
         const unsigned leader = __ffs(m) - 1;
         unsigned long long b = 0;
         if (lane_id() == leader) {
-            b = atomicAdd(&a.ctr[kQ + 8 * (k & 1) + qTail], (unsigned long long)__popc(m));
-            atomicAdd(&a.ctr[kQ + 8 * (k & 1) + qEval], (unsigned long long)__popc(m));
+            b = atomicAdd(QC(a, k & 1, qTail), (unsigned long long)__popc(m));
+            atomicAdd(QC(a, k & 1, qEval), (unsigned long long)__popc(m));
         }
         b = __shfl_sync(kFull, b, leader);
         if (wk)
@@ -571,21 +582,24 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
         if (gtid == 0 && (int64_t)k < a.nk_cap) a.nk[k] = (int64_t)rem;
         if (rem == 0 || k >= a.max_rounds) break;
         if (a.ctr[kErrPar + ((k - 1) & 1)] != 0) break;  // a trap fired (grid-uniform)
-        unsigned long long *qs = a.ctr + kQ + 8 * (k & 1);
+        const int qset = (int)(k & 1);
         uint2 *Qk = a.Q[k & 1];
-        if (PROF && gtid == 0 && (int64_t)k < a.nk_cap) a.rstat[4 * k + 3] = (int64_t)qs[qTail];
-        // dynamic queue: claim, wait for publication, process, mark done
-        for (;;) {
+        if (PROF && gtid == 0 && (int64_t)k < a.nk_cap) a.rstat[4 * k + 3] = (int64_t)*QC(a, qset, qTail);
+        // dynamic queue: claim, wait for publication, process, mark done.
+        // A round has ~10^4 items; kDynWarps warps are plenty, the others go
+        // straight to the barrier instead of polling the queue counters.
+        for (; gwarp < kDynWarps;) {
             unsigned long long idx = 0;
-            if (lane == 0) idx = atomicAdd(&qs[qHead], 1ull);
+            if (lane == 0) idx = atomicAdd(QC(a, qset, qHead), 1ull);
             idx = __shfl_sync(kFull, idx, 0);
             unsigned ix = 0, iy = 0;
             int state = 0;  // 1: item, 2: phase over, 3: timeout / abort
             if (lane == 0) {
                 const unsigned long long tw0 = gtimer();
+                unsigned backoff = 32;
                 for (;;) {
-                    const unsigned long long d = ld_acquire(&qs[qDone]);
-                    const unsigned long long t = ld_acquire(&qs[qTail]);
+                    const unsigned long long d = ld_acquire(QC(a, qset, qDone));
+                    const unsigned long long t = ld_acquire(QC(a, qset, qTail));
                     if (idx < t) {
                         volatile uint2 *src = reinterpret_cast<volatile uint2 *>(&Qk[idx]);
                         while ((iy = src->y) == 0u)
@@ -604,7 +618,8 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
                         state = 3;
                         break;
                     }
-                    __nanosleep(20);
+                    __nanosleep(backoff);
+                    backoff = min(backoff * 2u, 1024u);
                 }
             }
             state = __shfl_sync(kFull, state, 0);
@@ -622,12 +637,12 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
             if (lane == 0) {
                 Qk[idx] = make_uint2(0u, 0u);  // clean slot for the round after next
                 __threadfence();
-                atomicAdd(&qs[qDone], 1ull);
+                atomicAdd(QC(a, qset, qDone), 1ull);
             }
         }
         if (PROF && gtid == 0 && (int64_t)k < a.nk_cap) {
-            a.rstat[4 * k] = (int64_t)qs[qEval];
-            a.rstat[4 * k + 2] = (int64_t)qs[qLS];
+            a.rstat[4 * k] = (int64_t)*QC(a, qset, qEval);
+            a.rstat[4 * k + 2] = (int64_t)*QC(a, qset, qLS);
         }
         // the next phase pushes its NOTIFY items into set (k+2)&1 == k&1: reset it
         if (!grid_barrier(a, 3, k, (int)(k & 1))) return;
@@ -683,6 +698,8 @@ int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     if (rc) return rc;
     GC_CUDA_TRY(cudaMemsetAsync(s.S, 0, sizeof(uint32_t) * (size_t)n, g->stream));
     GC_CUDA_TRY(cudaMemsetAsync(s.ctr, 0, 64 * sizeof(unsigned long long), g->stream));
+    if (!s.qctl) GC_CUDA_TRY(cudaMalloc(&s.qctl, 256 * sizeof(unsigned long long)));
+    GC_CUDA_TRY(cudaMemsetAsync(s.qctl, 0, 256 * sizeof(unsigned long long), g->stream));
     // per-round queue: NOTIFY items (<= n + m/128) + EVAL (<= n) + SCAN (<= n + m/256)
     const size_t qcap = (size_t)(3 * n + g->nnz / 64 + 64);
     if (s.Qd[0] == nullptr || s.qd_cap < qcap) {
@@ -714,6 +731,7 @@ int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     a.SQ0 = reinterpret_cast<uint2 *>(s.Q2);
     a.LS = reinterpret_cast<LongScan *>(s.LS);
     a.Q[0] = reinterpret_cast<uint2 *>(s.Qd[0]);
+    a.qc = s.qctl;
     a.Q[1] = reinterpret_cast<uint2 *>(s.Qd[1]);
     a.ctr = s.ctr;
     a.nk = s.nk;
