@@ -320,6 +320,10 @@ __device__ __forceinline__ void eval_warp(const Args &a, uint32_t v, uint32_t k,
                 __threadfence();
             }
         }
+        // every lane publishes SCAN items that point at the slot lane 0 just
+        // wrote: __syncwarp orders that store before the lanes' own (fenced)
+        // item stores, so a consumer that sees an item sees the slot
+        __syncwarp();
         slot = __shfl_sync(kFull, slot, 0);
         if (slot == ~0ull) return;
         if (stat) {
