@@ -312,7 +312,7 @@ __device__ __forceinline__ void eval_warp(const Args &a, uint32_t v, uint32_t k,
                 L.ticket = nseg;
                 L.minH = f.hpos >= 0 ? (uint32_t)(f.hpos - rs) : kNone;
                 L.minL = f.lpos >= 0 ? (uint32_t)(f.lpos - rs) : kNone;
-                L.need = (miss_hi ? 1u : 0u) | (miss_lo ? 2u : 0u);
+                L.need = (miss_hi ? 1u : 0u) | (miss_lo ? 2u : 0u) | (k << 2);  // + round tag
                 L.sh = (uint32_t)(r.sh - rs);
                 L.sl = (uint32_t)(r.sl - rs);
                 L.base = (uint32_t)(lim - rs);
@@ -364,6 +364,10 @@ __device__ __forceinline__ void scan_segment(const Args &a, uint32_t slot, uint3
     const uint32_t v = __ldcg(&L->v);
     const uint32_t need = __ldcg(&L->need);
     const uint32_t Lbase = __ldcg(&L->base), Lsh = __ldcg(&L->sh), Lsl = __ldcg(&L->sl);
+    if ((need >> 2) != k) {  // trap: slot written by another round
+        if (lane == 0) flag_error(a, 15, k, (need >> 2));
+        return;
+    }
     if (v >= (uint32_t)a.n) {
         if (lane == 0) flag_error(a, 11, k, v);
         return;
