@@ -432,7 +432,12 @@ __device__ __forceinline__ void scan_segment(const Args &a, uint32_t slot, uint3
         const uint32_t mH = atomicAdd(&L->minH, 0u), mL = atomicAdd(&L->minL, 0u);
         const uint32_t deg = (uint32_t)(re - rs);
         const bool bad = (mH != kNone && mH >= deg) || (mL != kNone && mL >= deg);
-        if (bad) flag_error(a, 13, k, v);
+        if (bad) {
+            flag_error(a, (mH != kNone && mH >= deg) ? 13 : 14, k, v);
+            a.ctr[47] = deg;
+            a.ctr[48] = ((unsigned long long)mH << 32) | mL;
+            a.ctr[49] = ((unsigned long long)Lbase << 32) | (need & 3u);
+        }
         const Resume r = resume_of(v, rs, dense, a.W, a.P, a.C, thresh);
         Found f;
         if (mH != kNone && !bad) {
@@ -768,8 +773,9 @@ int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
     if (h[kErr - kRem] != 0) {
         char buf[160];
-        snprintf(buf, sizeof(buf), "internal consistency check %llu failed in round %llu (%llu)",
-                 h[kErr - kRem], h[kErr - kRem + 1], h[kErr - kRem + 2]);
+        snprintf(buf, sizeof(buf),
+                 "internal consistency check %llu failed in round %llu (%llu) dbg %llu %llx %llx",
+                 h[kErr - kRem], h[kErr - kRem + 1], h[kErr - kRem + 2], h[7], h[8], h[9]);
         set_error(buf);
         return GC_ERR_CUDA;
     }
