@@ -105,6 +105,7 @@ struct Args {
     uint32_t key;
     uint32_t max_rounds;
     unsigned long long q_cap, sq_cap, ls_cap;
+    unsigned long long dyn_warps;  // warps serving the dynamic queue
 };
 
 // Queue counters live on separate 128-byte lines: idle warps poll qDone/qTail
@@ -601,7 +602,7 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
         // dynamic queue: claim, wait for publication, process, mark done.
         // A round has ~10^4 items; kDynWarps warps are plenty, the others go
         // straight to the barrier instead of polling the queue counters.
-        for (; gwarp < kDynWarps;) {
+        for (; gwarp < a.dyn_warps;) {
             unsigned long long idx = 0;
             if (lane == 0) idx = atomicAdd(QC(a, qset, qHead), 1ull);
             idx = __shfl_sync(kFull, idx, 0);
@@ -756,6 +757,7 @@ int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     a.q_cap = (unsigned long long)qcap;
     a.sq_cap = (unsigned long long)(n + g->nnz / 128 + 1);
     a.ls_cap = (unsigned long long)n;
+    a.dyn_warps = p.dyn_warps > 0 ? (unsigned long long)p.dyn_warps : kDynWarps;
     const bool prof = p.prof && p.prof->on;
     cudaEvent_t e0 = nullptr, e1 = nullptr;
     if (prof) {
