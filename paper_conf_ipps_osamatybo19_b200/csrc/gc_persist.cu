@@ -423,7 +423,9 @@ __device__ __forceinline__ void scan_segment(const Args &a, uint32_t slot, uint3
     bool last = false;
     if (lane == 0) {
         __threadfence();
-        last = atomicSub(&L->ticket, 1u) == 1u;
+        const uint32_t old = atomicSub(&L->ticket, 1u);
+        if (old == 0u || old > 0x7FFFFFFFu) flag_error(a, 41, k, v);
+        last = old == 1u;
     }
     last = __shfl_sync(kFull, last, 0);
     if (!last) return;
@@ -498,8 +500,13 @@ __device__ __forceinline__ void process_item(const Args &a, uint2 it, uint32_t k
     const uint32_t type = it.y >> 28, sub = it.y & kSub;
     const unsigned lane = lane_id();
     if (type == T_EVAL) {
+        if (lane == 0 && atomicAdd(&a.S[it.x], 0u) != k) flag_error(a, 40, k, it.x);
         eval_warp<PROF>(a, it.x, k, nvisE);
     } else if (type == T_SCAN) {
+        if (it.x >= *QC(a, k & 1, qLS)) {
+            if (lane == 0) flag_error(a, 42, k, it.x);
+            return;
+        }
         scan_segment<PROF>(a, it.x, sub, k, nvisS);
     } else if (type == T_NOTIFY) {
         const uint32_t u = it.x;
