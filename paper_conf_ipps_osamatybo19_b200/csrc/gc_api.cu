@@ -534,6 +534,7 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     p.eval_big_min = o->hub_deg_min > 0 ? o->hub_deg_min : 256;
     p.batch_rounds = o->batch_rounds;
     p.dyn_warps = o->reserved[0];  // reserved[0]: event-mode queue warps (debug / tuning)
+    p.split = o->reserved[1];      // reserved[1]: event-mode split notify sub-phase (debug)
     p.max_rounds = (int64_t)(0x7FFFFFFFll / (2 * H)) + 1;
     Profile prof;
     prof.on = (o->flags & GC_PROFILE) != 0;

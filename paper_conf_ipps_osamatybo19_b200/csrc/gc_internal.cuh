@@ -127,6 +127,7 @@ struct RunParams {
     int32_t eval_big_min = 256;  // event mode: remaining scan length sent to a CTA
     int32_t batch_rounds = 0;
     int32_t dyn_warps = 0;       // event mode: warps serving the dynamic queue (0: default)
+    int32_t split = 0;           // event mode debug: notify sub-phase before evaluation
     int64_t max_rounds = 0;
 };
 

@@ -106,6 +106,7 @@ struct Args {
     uint32_t max_rounds;
     unsigned long long q_cap, sq_cap, ls_cap;
     unsigned long long dyn_warps;  // warps serving the dynamic queue
+    int split;                     // debug: NOTIFY items in a static sub-phase first
 };
 
 // Queue counters live on separate 128-byte lines: idle warps poll qDone/qTail
@@ -606,12 +607,27 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
         const int qset = (int)(k & 1);
         uint2 *Qk = a.Q[k & 1];
         if (PROF && gtid == 0 && (int64_t)k < a.nk_cap) a.rstat[4 * k + 3] = (int64_t)*QC(a, qset, qTail);
+        unsigned long long base0 = 0;  // first index served by the dynamic loop
+        if (a.split) {
+            // debug / A-B: the NOTIFY(k-1) items (the static prefix) first,
+            // statically, then a barrier, then the EVAL / SCAN items they made
+            const unsigned long long ns = *QC(a, qset, qTail);
+            for (unsigned long long i = gwarp; i < ns; i += nwarps) {
+                volatile uint2 *src = reinterpret_cast<volatile uint2 *>(&Qk[i]);
+                const uint2 it = make_uint2(src->x, src->y);
+                process_item<PROF>(a, it, k, nvisE, nvisS, nvisN);
+                __syncwarp();
+                if (lane == 0) Qk[i] = make_uint2(0u, 0u);
+            }
+            if (!grid_barrier(a, 4, k, -1)) return;
+            base0 = ns;
+        }
         // dynamic queue: claim, wait for publication, process, mark done.
         // A round has ~10^4 items; kDynWarps warps are plenty, the others go
         // straight to the barrier instead of polling the queue counters.
         for (; gwarp < a.dyn_warps;) {
             unsigned long long idx = 0;
-            if (lane == 0) idx = atomicAdd(QC(a, qset, qHead), 1ull);
+            if (lane == 0) idx = base0 + atomicAdd(QC(a, qset, qHead), 1ull);
             idx = __shfl_sync(kFull, idx, 0);
             unsigned ix = 0, iy = 0;
             int state = 0;  // 1: item, 2: phase over, 3: timeout / abort
@@ -630,7 +646,7 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
                         state = iy ? 1 : 3;
                         break;
                     }
-                    if (d == t) {
+                    if (d + base0 == t) {
                         state = 2;
                         break;
                     }
@@ -765,6 +781,7 @@ int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     a.sq_cap = (unsigned long long)(n + g->nnz / 128 + 1);
     a.ls_cap = (unsigned long long)n;
     a.dyn_warps = p.dyn_warps > 0 ? (unsigned long long)p.dyn_warps : kDynWarps;
+    a.split = p.split;
     const bool prof = p.prof && p.prof->on;
     cudaEvent_t e0 = nullptr, e1 = nullptr;
     if (prof) {
