@@ -297,6 +297,8 @@ __device__ __forceinline__ void eval_warp(const Args &a, uint32_t v, uint32_t k,
     warp_search(a.ci, a.C, thresh, a.key, weight_mix(v ^ a.key), r.need_hi, r.need_lo, r.sh, r.sl,
                 lim, f, vis);
     if (PROF) nvis += vis;
+    if (lane == 0 && f.hpos >= 0 && (f.hpos < s || f.hpos >= lim)) flag_error(a, 50, k, v);
+    if (lane == 0 && f.lpos >= 0 && (f.lpos < s || f.lpos >= lim)) flag_error(a, 51, k, v);
     const bool miss_hi = r.need_hi && f.hpos < 0;
     const bool miss_lo = r.need_lo && f.lpos < 0;
     if (lim < re && (miss_hi || miss_lo)) {
@@ -318,8 +320,13 @@ __device__ __forceinline__ void eval_warp(const Args &a, uint32_t v, uint32_t k,
                 L.sh = (uint32_t)(r.sh - rs);
                 L.sl = (uint32_t)(r.sl - rs);
                 L.base = (uint32_t)(lim - rs);
+                if ((L.minH != kNone && L.minH >= (uint32_t)(re - rs)) ||
+                    (L.minL != kNone && L.minL >= (uint32_t)(re - rs)))
+                    flag_error(a, 52, k, v);
                 a.LS[slot] = L;
                 __threadfence();
+                if (__ldcg(&a.LS[slot].minL) != L.minL || __ldcg(&a.LS[slot].v) != v)
+                    flag_error(a, 53, k, v);
             }
         }
         // every lane publishes SCAN items that point at the slot lane 0 just
