@@ -106,6 +106,7 @@ struct Args {
     uint32_t max_rounds;
     unsigned long long q_cap, sq_cap, ls_cap;
     unsigned long long dyn_warps;  // warps serving the dynamic queue
+    uint32_t *owner;               // debug: slot owner (round << 1 | busy)
     int split;                     // debug: NOTIFY items in a static sub-phase first
 };
 
@@ -307,6 +308,10 @@ __device__ __forceinline__ void eval_warp(const Args &a, uint32_t v, uint32_t k,
         unsigned long long slot = 0;
         if (lane == 0) {
             slot = atomicAdd(lsc, 1ull);
+            if (slot < a.ls_cap) {
+                const uint32_t prev = atomicExch(&a.owner[slot], (k << 1) | 1u);
+                if (prev == ((k << 1) | 1u)) flag_error(a, 60, k, (uint32_t)slot);
+            }
             if (slot >= a.ls_cap) {
                 flag_error(a, 2, k, v);
                 slot = ~0ull;
@@ -461,6 +466,7 @@ __device__ __forceinline__ void scan_segment(const Args &a, uint32_t slot, uint3
         }
         if (a.C[v] != GC_UNC) flag_error(a, 4, k, v);
         if (!bad) colored = settle(v, rs, r, f, k, a.C, a.W, a.P);
+        atomicExch(&a.owner[slot], k << 1);
     }
     colored = __shfl_sync(kFull, colored, 0);
     colored_notify(a, colored && lane == 0, v, re - rs, k, !colored && lane == 0);
@@ -789,6 +795,8 @@ int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     a.ls_cap = (unsigned long long)n;
     a.dyn_warps = p.dyn_warps > 0 ? (unsigned long long)p.dyn_warps : kDynWarps;
     a.split = p.split;
+    a.owner = s.Q3;
+    GC_CUDA_TRY(cudaMemsetAsync(s.Q3, 0, sizeof(uint32_t) * (size_t)n, g->stream));
     const bool prof = p.prof && p.prof->on;
     cudaEvent_t e0 = nullptr, e1 = nullptr;
     if (prof) {
