@@ -310,7 +310,10 @@ __device__ __forceinline__ void eval_warp(const Args &a, uint32_t v, uint32_t k,
             slot = atomicAdd(lsc, 1ull);
             if (slot < a.ls_cap) {
                 const uint32_t prev = atomicExch(&a.owner[slot], (k << 1) | 1u);
-                if (prev == ((k << 1) | 1u)) flag_error(a, 60, k, (uint32_t)slot);
+                if (prev & 1u) {  // still busy: same round (60) or an earlier one (61)
+                    flag_error(a, (prev >> 1) == k ? 60 : 61, k, (uint32_t)slot);
+                    a.ctr[47] = prev >> 1;
+                }
             }
             if (slot >= a.ls_cap) {
                 flag_error(a, 2, k, v);
