@@ -353,8 +353,13 @@ __device__ __forceinline__ void eval_warp(const Args &a, uint32_t v, uint32_t k,
             }
             for (uint32_t i = lane; i < nseg; i += 32) a.SQ0[b + i] = make_uint2((uint32_t)slot, i);
         } else {
-            push_items(a, k & 1, nseg, k,
-                       [&](uint32_t i) { return make_uint2((uint32_t)slot, (T_SCAN << 28) | i); });
+            // lane 0 wrote the slot, so lane 0 publishes its items: the slot
+            // store is then ordered before every item by lane 0's own fences
+            if (lane == 0) {
+                const unsigned long long b = atomicAdd(QC(a, k & 1, qTail), (unsigned long long)nseg);
+                for (uint32_t i = 0; i < nseg; ++i)
+                    put_item(a, k & 1, b + i, make_uint2((uint32_t)slot, (T_SCAN << 28) | i), k);
+            }
         }
         return;
     }
