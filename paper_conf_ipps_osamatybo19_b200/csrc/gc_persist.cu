@@ -260,7 +260,7 @@ __device__ __forceinline__ void lane_window(const Args &a, uint32_t thresh, uint
 #pragma unroll
     for (int q = 0; q < WIN; ++q) u[q] = s + q < lim ? a.ci[s + q] : 0u;
 #pragma unroll
-    for (int q = 0; q < WIN; ++q) c[q] = s + q < lim ? a.C[u[q]] : 0u;
+    for (int q = 0; q < WIN; ++q) c[q] = s + q < lim ? __ldcg(&a.C[u[q]]) : 0u;
 #pragma unroll
     for (int q = 0; q < WIN; ++q) {
         const int64_t e = s + q;
@@ -417,7 +417,7 @@ __device__ __forceinline__ void scan_segment(const Args &a, uint32_t slot, uint3
 #pragma unroll
         for (int q = 0; q < kSeg / 32; ++q) {
             const int64_t e = e0 + q * 32 + lane;
-            c[q] = e < e1 ? a.C[u[q]] : 0u;
+            c[q] = e < e1 ? __ldcg(&a.C[u[q]]) : 0u;
         }
         uint32_t rh = kNone, rl = kNone;
 #pragma unroll
@@ -494,9 +494,9 @@ __device__ __forceinline__ void notify_entries(const Args &a, uint32_t u, int64_
         w[q] = e < re ? a.ci[e] : kNone;
     }
 #pragma unroll
-    for (int q = 0; q < Q; ++q) cw[q] = w[q] != kNone ? a.C[w[q]] : 0u;
+    for (int q = 0; q < Q; ++q) cw[q] = w[q] != kNone ? __ldcg(&a.C[w[q]]) : 0u;
 #pragma unroll
-    for (int q = 0; q < Q; ++q) ww[q] = cw[q] == GC_UNC ? a.W[w[q]] : make_uint2(kNone, kNone);
+    for (int q = 0; q < Q; ++q) ww[q] = cw[q] == GC_UNC ? __ldcg(&a.W[w[q]]) : make_uint2(kNone, kNone);
 #pragma unroll
     for (int q = 0; q < Q; ++q) {
         bool wk = cw[q] == GC_UNC && (ww[q].x == u || ww[q].y == u);
