@@ -176,7 +176,7 @@ class Graph:
     def color(self, seed: int = 1, variant: int = MAXMIN, out=None, *, flags: int = 0,
               mode: int = MODE_AUTO, batch_rounds: int = 0, thread_deg_max: int = 0,
               hub_deg_min: int = 0, stats: bool = False, frontier_cap: int = 0,
-              trace_cap: int = 0, dyn_warps: int = 0, split: int = 0):
+              trace_cap: int = 0):
         """Colour the graph.  `out`: int32 tensor/array of n entries on host or
         device (allocated on the host if None).  Returns (out, n_colors) or
         (out, n_colors, ColorStats) with stats=True."""
@@ -187,8 +187,6 @@ class Graph:
         o.struct_size = ctypes.sizeof(gc_options)
         o.variant, o.seed, o.flags, o.mode = variant, seed, flags, mode
         o.batch_rounds, o.thread_deg_max, o.hub_deg_min = batch_rounds, thread_deg_max, hub_deg_min
-        o.reserved[0] = dyn_warps
-        o.reserved[1] = split
         st = gc_stats()
         st.struct_size = ctypes.sizeof(gc_stats)
         fs = None

@@ -335,9 +335,6 @@ static void free_scratch(Scratch &s) {
     cudaFree(s.Q2);
     cudaFree(s.Q3);
     cudaFree(s.LS);
-    cudaFree(s.Qd[0]);
-    cudaFree(s.Qd[1]);
-    cudaFree(s.qctl);
     cudaFree(s.ctr);
     cudaFree(s.nk);
     cudaFree(s.rstat);
@@ -533,8 +530,6 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     p.hub_deg_min = o->hub_deg_min > 0 ? o->hub_deg_min : 4096;
     p.eval_big_min = o->hub_deg_min > 0 ? o->hub_deg_min : 256;
     p.batch_rounds = o->batch_rounds;
-    p.dyn_warps = o->reserved[0];  // reserved[0]: event-mode queue warps (debug / tuning)
-    p.split = o->reserved[1];      // reserved[1]: event-mode split notify sub-phase (debug)
     p.max_rounds = (int64_t)(0x7FFFFFFFll / (2 * H)) + 1;
     Profile prof;
     prof.on = (o->flags & GC_PROFILE) != 0;

@@ -54,8 +54,8 @@ __device__ __forceinline__ void warp_search(const uint32_t *__restrict__ ci, con
         const int64_t e1 = e0 + lane, e2 = e0 + 32 + lane;
         const uint32_t u1 = e1 < re ? ci[e1] : 0u;
         const uint32_t u2 = e2 < re ? ci[e2] : 0u;
-        const uint32_t c1 = e1 < re ? __ldcg(&C[u1]) : 0u;
-        const uint32_t c2 = e2 < re ? __ldcg(&C[u2]) : 0u;
+        const uint32_t c1 = e1 < re ? C[u1] : 0u;
+        const uint32_t c2 = e2 < re ? C[u2] : 0u;
         nvis += (e1 < re) + (e2 < re);
         bool h1 = false, l1 = false, h2 = false, l2 = false;
         if (e1 < re && c1 >= thresh) {
@@ -109,10 +109,10 @@ __device__ __forceinline__ Resume resume_of(uint32_t v, int64_t rs, bool dense, 
         r.need_hi = r.need_lo = true;
         r.sh = r.sl = rs;
     } else {
-        const uint2 w = __ldcg(&W[v]);
-        const uint2 p = __ldcg(&P[v]);
-        r.need_hi = __ldcg(&C[w.x]) < thresh;  // hi witness coloured in an earlier round
-        r.need_lo = __ldcg(&C[w.y]) < thresh;
+        const uint2 w = W[v];
+        const uint2 p = P[v];
+        r.need_hi = C[w.x] < thresh;  // hi witness coloured in an earlier round
+        r.need_lo = C[w.y] < thresh;
         r.sh = rs + (int64_t)p.x + 1;
         r.sl = rs + (int64_t)p.y + 1;
     }

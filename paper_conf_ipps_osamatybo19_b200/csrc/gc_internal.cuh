@@ -49,9 +49,6 @@ struct Scratch {
     uint32_t *Q2 = nullptr;       // event mode: long-row notify / long-scan segment queue
     uint32_t *Q3 = nullptr;       // persistent event mode: notify segment queue
     void *LS = nullptr;           // persistent event mode: long-scan slots (32 B each)
-    void *Qd[2] = {nullptr, nullptr};  // persistent event mode: per-round work queues
-    size_t qd_cap = 0;
-    unsigned long long *qctl = nullptr;  // persistent event mode: queue counters
     uint32_t *S = nullptr;        // Luby inner-loop state / event stamps
     uint32_t *W = nullptr;        // event mode: witness pairs (2 per vertex)
     uint32_t *P = nullptr;        // event mode: resume cursors (2 per vertex)
@@ -126,8 +123,6 @@ struct RunParams {
     int32_t hub_deg_min = 4096;
     int32_t eval_big_min = 256;  // event mode: remaining scan length sent to a CTA
     int32_t batch_rounds = 0;
-    int32_t dyn_warps = 0;       // event mode: warps serving the dynamic queue (0: default)
-    int32_t split = 0;           // event mode debug: notify sub-phase before evaluation
     int64_t max_rounds = 0;
 };
 
