@@ -279,8 +279,8 @@ def main():
         torch.cuda.synchronize()
         peak, peak_src = measured_peaks()
         cls = max(range(4), key=lambda c: sp.kernel_ms[c])
-        names = {gcb.MODE_EVENT: {0: "k_event_persistent", 1: "round 0 (static phases)",
-                                  2: "rounds >= 1 (one dynamic-queue phase each)", 3: "-"},
+        names = {gcb.MODE_EVENT: {0: "k_event_persistent", 1: "phase P1 eval (all rounds)",
+                                  2: "phase P1b+P2 long scans", 3: "phase P3 notify"},
                  gcb.MODE_EVENT_MULTI: {0: "k_eval", 1: "k_eval_big", 2: "k_notify",
                                         3: "k_notify_big"},
                  gcb.MODE_SWEEP: {0: "k_sweep", 1: "k_hub", 2: "other", 3: "other"}}[sp.mode_used]
