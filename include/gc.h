@@ -131,9 +131,10 @@ typedef struct gc_stats {
     int64_t kernel_bytes[4];
     int64_t visits;
     /* GC_PROFILE only, optional caller buffers: the duration of every timed
-     * launch in launch order (us), and per round 4 counters (event mode:
-     * |D_k| evaluated, |I_k| coloured, long scans, long-row notify items;
-     * sweep mode: N_k, hubs, 0, 0). */
+     * launch in launch order (us), and per round 8 values (event mode:
+     * |D_k| evaluated, |I_k| coloured, long scans, long-row notify items,
+     * then the persistent kernel's P1 / P1b+P2 / P3 phase times in ns;
+     * sweep mode: N_k, 0...). */
     float *launch_us;
     int64_t launch_cap;
     int64_t *round_stats;

@@ -412,7 +412,7 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
             for (int i = 0; i < 8; ++i) cn[i] = 0;
             if (PROF) {
                 a.ctr[kSumD] += N;
-                if ((int64_t)k < a.nk_cap) a.rstat[4 * k] = (int64_t)N;
+                if ((int64_t)k < a.nk_cap) a.rstat[8 * k] = (int64_t)N;
                 t0 = gtimer();
             }
         }
@@ -458,6 +458,7 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
         if (PROF && gtid == 0) {
             unsigned long long t = gtimer();
             tacc[0] += t - t0;
+            if ((int64_t)k < a.nk_cap) a.rstat[8 * k + 4] = (int64_t)(t - t0);
             t0 = t;
         }
         // ----------------------------------------------------------- P1b
@@ -477,6 +478,7 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
         if (PROF && gtid == 0) {
             unsigned long long t = gtimer();
             tacc[1] += t - t0;
+            if ((int64_t)k < a.nk_cap) a.rstat[8 * k + 5] = (int64_t)(t - t0);
             t0 = t;
         }
         // ------------------------------------------------------------ P3
@@ -506,15 +508,16 @@ __global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
             if (PROF && lane == 0) nvisN += (uint32_t)(re - rs);
         }
         if (PROF && gtid == 0 && (int64_t)k < a.nk_cap) {
-            a.rstat[4 * k + 1] = (int64_t)ncol;
-            a.rstat[4 * k + 2] = (int64_t)cs[cLS];
-            a.rstat[4 * k + 3] = (int64_t)nq;
+            a.rstat[8 * k + 1] = (int64_t)ncol;
+            a.rstat[8 * k + 2] = (int64_t)cs[cLS];
+            a.rstat[8 * k + 3] = (int64_t)nq;
         }
         rem -= ncol;
         if (!phase_barrier(a, 3, k)) return;
         if (PROF && gtid == 0) {
             unsigned long long t = gtimer();
             tacc[2] += t - t0;
+            if ((int64_t)k < a.nk_cap) a.rstat[8 * k + 6] = (int64_t)(t - t0);
             t0 = t;
         }
     }

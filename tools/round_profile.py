@@ -23,19 +23,20 @@ def main():
     ap.add_argument("--out", default="gpurun_out/rounds.json")
     a = ap.parse_args()
     g = G.rmat(a.scale, 16, seed=1, device="cuda")
-    mode = {"event": gcb.MODE_EVENT, "sweep": gcb.MODE_SWEEP}[a.mode]
+    mode = {"event": gcb.MODE_EVENT, "sweep": gcb.MODE_SWEEP, "multi": gcb.MODE_EVENT_MULTI}[a.mode]
     out = torch.empty(g.n, dtype=torch.int32, device="cuda")
     with gcb.Graph(g.n, g.row_offsets, g.col_indices, flags=gcb.BORROW_DEVICE) as h:
         h.color(1, gcb.MAXMIN, out, mode=mode)
         _, k, st = h.color(1, gcb.MAXMIN, out, mode=mode, flags=gcb.PROFILE, stats=True,
                            trace_cap=1 << 15)
     R = st.rounds
-    per = 4 if mode == gcb.MODE_EVENT else 2
+    per = {gcb.MODE_EVENT: 3, gcb.MODE_EVENT_MULTI: 4}.get(mode, 2)
     lu = st.launch_us
     rows = []
     for r in range(R):
-        t = lu[per * r: per * r + per]
-        rs = st.round_stats[4 * r: 4 * r + 4]
+        rs = st.round_stats[8 * r: 8 * r + 8]
+        # persistent kernel: per-phase times (ns) are in the round record
+        t = [x / 1e3 for x in rs[4:7]] if mode == gcb.MODE_EVENT else lu[per * r: per * r + per]
         rows.append({"k": r, "us": t, "stats": rs})
     buckets = [(0, 1), (1, 2), (2, 10), (10, 100), (100, 500), (500, 1000), (1000, 2000),
                (2000, R)]
@@ -45,7 +46,7 @@ def main():
         if not sel:
             continue
         tot = [sum(x["us"][c] for x in sel) for c in range(per)]
-        st4 = [sum(x["stats"][c] for x in sel) for c in range(4)]
+        st4 = [sum(x["stats"][c] for x in sel) for c in range(8)]
         summ.append({"rounds": [lo, min(hi, R)], "us_by_class": tot, "us_total": sum(tot),
                      "stat_sums": st4, "us_per_round": sum(tot) / len(sel)})
     res = {"scale": a.scale, "mode": a.mode, "rounds": R, "n_colors": k, "ms": st.ms,
