@@ -33,7 +33,7 @@ namespace {
 
 using namespace ev;
 
-constexpr int kThreads = 512;
+constexpr int kThreads = 1024;  // one block per SM: fewer barrier arrivals
 constexpr int kLaneWin = 8;      // entries a lane scans before handing off
 constexpr int kWarpWin = 256;    // entries a warp scans before splitting
 constexpr int kSeg = 256;        // entries per long-scan segment (8 per lane)
@@ -109,9 +109,9 @@ __device__ __forceinline__ unsigned long long gtimer() {
 // block is resident).  Generation barrier on ctr[kBar], ctr[kBar+1]: the last
 // block to arrive resets the count and bumps the generation.  A wait longer
 // than kBarrierTimeoutNs records a trap and makes every block leave the
-// kernel (returns false) instead of hanging the GPU.  Every thread then
-// issues a gpu-scope fence: the next phase reads state other SMs wrote (L1 is
-// not coherent; the fence invalidates it).
+// kernel (returns false) instead of hanging the GPU.  The waiting thread then
+// issues a gpu-scope fence, which also invalidates its SM's L1 (CCTL.IVALL):
+// the next phase reads state other SMs wrote, and L1 is not coherent.
 enum : int { kBar = 61, kAbort = 63 };
 constexpr unsigned long long kBarrierTimeoutNs = 4000000000ull;
 
@@ -145,11 +145,10 @@ __device__ __forceinline__ bool phase_barrier(const Args &a, int id, uint32_t k)
                 __nanosleep(64);
             }
         }
-        __threadfence();
+        __threadfence();  // gpu-scope fence after the wait: also invalidates this SM's L1
         ok_sh = ok;
     }
     __syncthreads();
-    __threadfence();
     return ok_sh != 0;
 }
 
@@ -378,10 +377,12 @@ __device__ __forceinline__ void notify_entries(const Args &a, uint32_t u, int64_
         const int64_t e = e0 + (int64_t)q * stride;
         w[q] = (u != kNone && e < re) ? a.ci[e] : kNone;
     }
+    // colour and witnesses are loaded together (one dependent step, not two)
 #pragma unroll
-    for (int q = 0; q < Q; ++q) cw[q] = w[q] != kNone ? a.C[w[q]] : 0u;
-#pragma unroll
-    for (int q = 0; q < Q; ++q) ww[q] = cw[q] == GC_UNC ? a.W[w[q]] : make_uint2(kNone, kNone);
+    for (int q = 0; q < Q; ++q) {
+        cw[q] = w[q] != kNone ? a.C[w[q]] : 0u;
+        ww[q] = w[q] != kNone ? a.W[w[q]] : make_uint2(kNone, kNone);
+    }
 #pragma unroll
     for (int q = 0; q < Q; ++q) {
         bool wk = cw[q] == GC_UNC && (ww[q].x == u || ww[q].y == u);
@@ -391,7 +392,7 @@ __device__ __forceinline__ void notify_entries(const Args &a, uint32_t u, int64_
 }
 
 template <bool PROF>
-__global__ void __launch_bounds__(kThreads, 2) k_event_persistent(Args a) {
+__global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
     const unsigned lane = lane_id();
     const unsigned long long gtid = (unsigned long long)blockIdx.x * blockDim.x + threadIdx.x;
     const unsigned long long nthreads = (unsigned long long)gridDim.x * blockDim.x;
