@@ -106,8 +106,7 @@ __device__ __forceinline__ unsigned long long gtimer() {
 }
 
 // Grid-wide phase boundary (the kernel is launched cooperatively, so every
-// block is resident).  Generation barrier on ctr[kBar], ctr[kBar+1]: the last
-// block to arrive resets the count and bumps the generation.  A wait longer
+// block is resident).  Monotone arrival counter on ctr[kBar].  A wait longer
 // than kBarrierTimeoutNs records a trap and makes every block leave the
 // kernel (returns false) instead of hanging the GPU.  The waiting thread then
 // issues a gpu-scope fence, which also invalidates its SM's L1 (CCTL.IVALL):
@@ -115,24 +114,27 @@ __device__ __forceinline__ unsigned long long gtimer() {
 enum : int { kBar = 61, kAbort = 63 };
 constexpr unsigned long long kBarrierTimeoutNs = 4000000000ull;
 
+__device__ __forceinline__ unsigned long long ld_acquire(const unsigned long long *p) {
+    unsigned long long v;
+    asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+    return v;
+}
+
 __device__ __forceinline__ bool phase_barrier(const Args &a, int id, uint32_t k) {
     __shared__ int ok_sh;
     __syncthreads();
     if (threadIdx.x == 0) {
+        // monotone arrival counter: barrier instance i completes when it
+        // reaches (i + 1) * gridDim.x -- one atomic per block, no reset
         int ok = 1;
-        volatile unsigned long long *gen = a.ctr + kBar + 1;
-        volatile unsigned long long *abort = a.ctr + kAbort;
-        const unsigned long long g0 = *gen;
         __threadfence();
-        const unsigned long long arrived = atomicAdd(a.ctr + kBar, 1ull) + 1;
-        if (arrived == gridDim.x) {
-            a.ctr[kBar] = 0;
-            __threadfence();
-            atomicAdd(a.ctr + kBar + 1, 1ull);
-        } else {
-            const unsigned long long t0 = gtimer();
-            while (*gen == g0) {
-                if (*abort) {
+        const unsigned long long old = atomicAdd(a.ctr + kBar, 1ull);
+        const unsigned long long target = (old / gridDim.x + 1) * gridDim.x;
+        unsigned spins = 0;
+        const unsigned long long t0 = gtimer();
+        while (ld_acquire(a.ctr + kBar) < target) {
+            if ((++spins & 255u) == 0u) {
+                if (*(volatile unsigned long long *)(a.ctr + kAbort)) {
                     ok = 0;
                     break;
                 }
@@ -142,7 +144,6 @@ __device__ __forceinline__ bool phase_barrier(const Args &a, int id, uint32_t k)
                     ok = 0;
                     break;
                 }
-                __nanosleep(64);
             }
         }
         __threadfence();  // gpu-scope fence after the wait: also invalidates this SM's L1
@@ -152,31 +153,106 @@ __device__ __forceinline__ bool phase_barrier(const Args &a, int id, uint32_t k)
     return ok_sh != 0;
 }
 
+// ---------------------------------------------------------------- staging
+// Appends to the shared lists (coloured rows to notify, woken vertices,
+// overflowing lane windows) and the coloured count are staged per block in
+// shared memory and flushed with ONE global atomic per list per block at the
+// end of each phase: with a warp per vertex every colouring would otherwise
+// be 2-3 global atomics on one cache line, serialised in one L2 slice.  A
+// list that overflows its shared buffer falls back to global appends.
+constexpr int kStNQS = 4096, kStNQ = 4096, kStD = 8192, kStWQ = 4096;
+struct Stage {
+    uint32_t nqs[kStNQS];
+    uint2 nq[kStNQ];
+    uint32_t d[kStD];
+    uint32_t wq[kStWQ];
+    unsigned n[4];            // staged counts: 0 nqs, 1 nq, 2 d, 3 wq
+    unsigned colored;         // staged coloured count
+    unsigned long long base[4];
+};
+constexpr size_t kStageBytes = sizeof(Stage);
+
+__device__ __forceinline__ Stage &stage() {
+    extern __shared__ __align__(16) unsigned char smem_raw[];
+    return *reinterpret_cast<Stage *>(smem_raw);
+}
+
+// Whole warp converged: lanes with `pred` append make(lane) to staged list
+// `li` (shared buffer buf of capacity cap), spilling to the global list /
+// counter beyond the capacity.
+template <class T>
+__device__ __forceinline__ void stage_append(bool pred, T val, int li, T *buf, int cap, T *glist,
+                                             unsigned long long *gcount) {
+    const unsigned m = __ballot_sync(kFull, pred);
+    if (!m) return;
+    Stage &st = stage();
+    const unsigned lane = lane_id();
+    const unsigned leader = __ffs(m) - 1;
+    unsigned base = 0;
+    if (lane == leader) base = atomicAdd(&st.n[li], (unsigned)__popc(m));
+    base = __shfl_sync(kFull, base, leader);
+    const unsigned pos = base + __popc(m & ((1u << lane) - 1u));
+    const bool spill = pred && pos >= (unsigned)cap;
+    if (pred && !spill) buf[pos] = val;
+    const unsigned sm = __ballot_sync(kFull, spill);
+    if (sm) {
+        const unsigned sl = __ffs(sm) - 1;
+        unsigned long long gb = 0;
+        if (lane == sl) gb = atomicAdd(gcount, (unsigned long long)__popc(sm));
+        gb = __shfl_sync(kFull, gb, sl);
+        if (spill) glist[gb + __popc(sm & ((1u << lane) - 1u))] = val;
+    }
+}
+
+// Whole block, at the end of a phase: move the staged entries to the global
+// lists (one atomicAdd per non-empty list) and add the coloured count.
+__device__ __forceinline__ void stage_flush(const Args &a, unsigned long long *cs,
+                                            unsigned long long *dcount, uint32_t *Dout) {
+    Stage &st = stage();
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        unsigned long long *ctrs[4] = {&cs[cNQS], &cs[cNQ], dcount, &cs[cWQ]};
+        const int caps[4] = {kStNQS, kStNQ, kStD, kStWQ};
+        for (int i = 0; i < 4; ++i) {
+            const unsigned c = min(st.n[i], (unsigned)caps[i]);
+            st.n[i] = c;
+            st.base[i] = c ? atomicAdd(ctrs[i], (unsigned long long)c) : 0ull;
+        }
+        if (st.colored) atomicAdd(&cs[cI], (unsigned long long)st.colored);
+        st.colored = 0;
+    }
+    __syncthreads();
+    for (unsigned i = threadIdx.x; i < st.n[0]; i += blockDim.x) a.NQS[st.base[0] + i] = st.nqs[i];
+    for (unsigned i = threadIdx.x; i < st.n[1]; i += blockDim.x) a.NQ[st.base[1] + i] = st.nq[i];
+    for (unsigned i = threadIdx.x; i < st.n[2]; i += blockDim.x) Dout[st.base[2] + i] = st.d[i];
+    for (unsigned i = threadIdx.x; i < st.n[3]; i += blockDim.x) a.WQ[st.base[3] + i] = st.wq[i];
+    __syncthreads();
+    if (threadIdx.x < 4) st.n[threadIdx.x] = 0;
+    // (the barrier that follows starts with __syncthreads)
+}
+
 // Enqueue the notification work of lanes whose vertex was just coloured
 // (whole warp converged).  Short rows -> NQS (one lane each); long rows ->
 // NQ segments.
 __device__ __forceinline__ void enqueue_notify(const Args &a, unsigned long long *cs, bool colored,
                                                uint32_t u, int64_t deg, uint32_t k) {
+    Stage &st = stage();
     const bool shortrow = colored && deg <= kLaneNotify;
-    warp_append(shortrow, u, a.NQS, &cs[cNQS]);
+    stage_append<uint32_t>(shortrow, u, 0, st.nqs, kStNQS, a.NQS, &cs[cNQS]);
     unsigned lm = __ballot_sync(kFull, colored && !shortrow);
-    while (lm) {  // long rows: the whole warp writes the segment items
+    while (lm) {  // long rows: the whole warp stages the segment items
         const int src = __ffs(lm) - 1;
         lm &= lm - 1;
         const uint32_t uu = __shfl_sync(kFull, u, src);
         const int64_t dg = __shfl_sync(kFull, deg, src);
         const uint32_t nseg = (uint32_t)((dg + kNotifySeg - 1) / kNotifySeg);
-        unsigned long long b = 0;
-        if (lane_id() == 0) b = atomicAdd(&cs[cNQ], (unsigned long long)nseg);
-        b = __shfl_sync(kFull, b, 0);
-        if (b + nseg > a.nq_cap) {
-            if (lane_id() == 0) flag_error(a, 1, k, uu);
-            continue;
+        for (uint32_t q0 = 0; q0 < nseg; q0 += 32) {
+            const uint32_t q = q0 + lane_id();
+            stage_append<uint2>(q < nseg, make_uint2(uu, q), 1, st.nq, kStNQ, a.NQ, &cs[cNQ]);
         }
-        for (uint32_t q = lane_id(); q < nseg; q += 32) a.NQ[b + q] = make_uint2(uu, q);
     }
     const unsigned m = __ballot_sync(kFull, colored);
-    if (m && lane_id() == (unsigned)(__ffs(m) - 1)) atomicAdd(&cs[cI], (unsigned long long)__popc(m));
+    if (m && lane_id() == (unsigned)(__ffs(m) - 1)) atomicAdd(&st.colored, (unsigned)__popc(m));
 }
 
 // Whole-warp evaluation of one vertex of D_k (warp-uniform arguments): scan a
@@ -387,7 +463,7 @@ __device__ __forceinline__ void notify_entries(const Args &a, uint32_t u, int64_
     for (int q = 0; q < Q; ++q) {
         bool wk = cw[q] == GC_UNC && (ww[q].x == u || ww[q].y == u);
         if (wk) wk = atomicMax(&a.S[w[q]], k + 1u) < k + 1u;
-        warp_append(wk, w[q], Dout, dcount);
+        stage_append<uint32_t>(wk, w[q], 2, stage().d, kStD, Dout, dcount);
     }
 }
 
@@ -401,6 +477,12 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
     uint32_t nvisE = 0, nvisS = 0, nvisN = 0;
     unsigned long long t0 = 0, tacc[4] = {0, 0, 0, 0};
     uint32_t k = 0;
+    {
+        Stage &st = stage();
+        if (threadIdx.x < 4) st.n[threadIdx.x] = 0;
+        if (threadIdx.x == 0) st.colored = 0;
+        __syncthreads();
+    }
     for (;; ++k) {
         unsigned long long *cs = a.ctr + kSet + 8 * (k & 1);
         unsigned long long *cn = a.ctr + kSet + 8 * ((k + 1) & 1);
@@ -419,6 +501,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
         }
         const uint32_t *Din = a.D[k & 1];
         uint32_t *Dout = a.D[(k + 1) & 1];
+        unsigned long long *dcount = &cn[cD];
         const uint32_t thresh = 2u * k;
         // ------------------------------------------------------------ P1
         if (dense || N > 4 * nwarps) {
@@ -448,13 +531,14 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
                     if (a.C[v] != GC_UNC) flag_error(a, 5, k, v);
                     colored = settle(v, rs, r, f, k, a.C, a.W, a.P);
                 }
-                warp_append(unresolved, v, a.WQ, &cs[cWQ]);
+                stage_append<uint32_t>(unresolved, v, 3, stage().wq, kStWQ, a.WQ, &cs[cWQ]);
                 enqueue_notify(a, cs, colored, v, re - rs, k);
             }
         } else {
             for (unsigned long long i = gwarp; i < N; i += nwarps)
                 eval_warp<PROF>(a, cs, Din[i], k, false, nvisE);
         }
+        stage_flush(a, cs, dcount, Dout);
         if (!phase_barrier(a, 0, k)) return;
         if (PROF && gtid == 0) {
             unsigned long long t = gtimer();
@@ -467,6 +551,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
         if (nwq) {
             for (unsigned long long i = gwarp; i < nwq; i += nwarps)
                 eval_warp<PROF>(a, cs, a.WQ[i], k, dense, nvisE);
+            stage_flush(a, cs, dcount, Dout);
             if (!phase_barrier(a, 1, k)) return;
         }
         // ------------------------------------------------------------ P2
@@ -474,6 +559,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
         if (nsq) {
             for (unsigned long long i = gwarp; i < nsq; i += nwarps)
                 scan_segment<PROF>(a, cs, a.SQ[i], k, dense, nvisS);
+            stage_flush(a, cs, dcount, Dout);
             if (!phase_barrier(a, 2, k)) return;
         }
         if (PROF && gtid == 0) {
@@ -485,7 +571,6 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
         // ------------------------------------------------------------ P3
         const unsigned long long ncol = cs[cI];
         const unsigned long long nqs = cs[cNQS], nq = cs[cNQ];
-        unsigned long long *dcount = &cn[cD];
         // short rows: 4 rows per warp, 8 lanes per row, 4 entries per lane
         for (unsigned long long base = gwarp * 4; base < nqs; base += nwarps * 4) {
             const unsigned long long idx = base + (lane >> 3);
@@ -514,6 +599,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
             a.rstat[8 * k + 3] = (int64_t)nq;
         }
         rem -= ncol;
+        stage_flush(a, cs, dcount, Dout);
         if (!phase_barrier(a, 3, k)) return;
         if (PROF && gtid == 0) {
             unsigned long long t = gtimer();
@@ -543,8 +629,10 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
 template <bool PROF>
 int launch(gc_graph *g, Args &a, int *blocks_out) {
     int per_sm = 0;
+    GC_CUDA_TRY(cudaFuncSetAttribute(k_event_persistent<PROF>,
+                                     cudaFuncAttributeMaxDynamicSharedMemorySize, (int)kStageBytes));
     GC_CUDA_TRY(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_event_persistent<PROF>,
-                                                              kThreads, 0));
+                                                              kThreads, kStageBytes));
     if (per_sm < 1) {
         set_error("persistent event kernel cannot be resident");
         return GC_ERR_CUDA;
@@ -552,7 +640,7 @@ int launch(gc_graph *g, Args &a, int *blocks_out) {
     const int blocks = per_sm * g->sm_count;
     void *args[] = {&a};
     GC_CUDA_TRY(cudaLaunchCooperativeKernel((void *)k_event_persistent<PROF>, blocks, kThreads, args,
-                                            0, g->stream));
+                                            kStageBytes, g->stream));
     *blocks_out = blocks;
     return GC_OK;
 }
