@@ -131,9 +131,10 @@ typedef struct gc_stats {
     int64_t kernel_bytes[4];
     int64_t visits;
     /* GC_PROFILE only, optional caller buffers: the duration of every timed
-     * launch in launch order (us), and per round 8 values (event mode:
+     * launch in launch order (us), and per round 16 values (event mode:
      * |D_k| evaluated, |I_k| coloured, long scans, long-row notify items,
-     * then the persistent kernel's P1 / P1b+P2 / P3 phase times in ns;
+     * the persistent kernel's P1 / P1b+P2 / P3 phase times in ns, -, then
+     * the longest per-block work time of P1 / P1b / P2 / P3 in ns;
      * sweep mode: N_k, 0...). */
     float *launch_us;
     int64_t launch_cap;

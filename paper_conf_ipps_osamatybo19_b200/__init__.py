@@ -197,7 +197,7 @@ class Graph:
         lu = rs = None
         if trace_cap:
             lu = (ctypes.c_float * (4 * trace_cap))()
-            rs = (ctypes.c_int64 * (8 * trace_cap))()
+            rs = (ctypes.c_int64 * (16 * trace_cap))()
             st.launch_us, st.launch_cap = ctypes.cast(lu, ctypes.c_void_p), 4 * trace_cap
             st.round_stats, st.round_stats_cap = ctypes.cast(rs, ctypes.c_void_p), trace_cap
         r = _check(lib().gc_color_ex(self._h, ctypes.byref(o), _ptr(out, ("int32",)),
@@ -208,7 +208,7 @@ class Graph:
                                       st.launches, st.ms, nk, list(st.kernel_ms),
                                       list(st.kernel_launches), list(st.kernel_bytes), st.visits,
                                       list(lu[: min(4 * trace_cap, 4 * st.rounds + 8)]) if lu else [],
-                                      list(rs[: min(8 * trace_cap, 8 * st.rounds)]) if rs else [])
+                                      list(rs[: min(16 * trace_cap, 16 * st.rounds)]) if rs else [])
         return out, r
 
     def close(self) -> None:

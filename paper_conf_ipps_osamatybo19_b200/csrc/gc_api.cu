@@ -228,12 +228,12 @@ int ensure_nk(gc_graph *g, int64_t need) {
     int64_t cap = std::max<int64_t>(need * 2, 1 << 12);
     int64_t *nk = nullptr, *rstat = nullptr;
     GC_CUDA_TRY(cudaMalloc(&nk, sizeof(int64_t) * cap));
-    GC_CUDA_TRY(cudaMalloc(&rstat, sizeof(int64_t) * 8 * cap));
-    GC_CUDA_TRY(cudaMemsetAsync(rstat, 0, sizeof(int64_t) * 8 * cap, g->stream));
+    GC_CUDA_TRY(cudaMalloc(&rstat, sizeof(int64_t) * 16 * cap));
+    GC_CUDA_TRY(cudaMemsetAsync(rstat, 0, sizeof(int64_t) * 16 * cap, g->stream));
     if (s.nk) {
         GC_CUDA_TRY(cudaMemcpyAsync(nk, s.nk, sizeof(int64_t) * s.nk_cap, cudaMemcpyDeviceToDevice,
                                     g->stream));
-        GC_CUDA_TRY(cudaMemcpyAsync(rstat, s.rstat, sizeof(int64_t) * 8 * s.nk_cap,
+        GC_CUDA_TRY(cudaMemcpyAsync(rstat, s.rstat, sizeof(int64_t) * 16 * s.nk_cap,
                                     cudaMemcpyDeviceToDevice, g->stream));
         GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
         cudaFree(s.nk);
@@ -595,7 +595,7 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
             int64_t m = std::min<int64_t>(std::min<int64_t>(stats->round_stats_cap, res.rounds + 1),
                                           g->s.nk_cap);
             if (m > 0)
-                GC_CUDA_TRY(cudaMemcpy(stats->round_stats, g->s.rstat, sizeof(int64_t) * 8 * m,
+                GC_CUDA_TRY(cudaMemcpy(stats->round_stats, g->s.rstat, sizeof(int64_t) * 16 * m,
                                        cudaMemcpyDeviceToHost));
         }
         if (stats->frontier_sizes && stats->frontier_cap > 0 && !luby) {

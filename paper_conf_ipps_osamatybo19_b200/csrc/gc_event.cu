@@ -69,7 +69,7 @@ __global__ void __launch_bounds__(kBlock) k_eval(
         if ((int64_t)k < nk_cap) nk[k] = (int64_t)ctr[kRem];
         if (PROF) {
             ctr[kSumD] += N;
-            if ((int64_t)k < nk_cap) rstat[8 * k] = (int64_t)N;
+            if ((int64_t)k < nk_cap) rstat[16 * k] = (int64_t)N;
         }
     }
     const uint32_t thresh = 2u * k;
@@ -302,9 +302,9 @@ __global__ void __launch_bounds__(kBlock) k_notify_big(
     const unsigned long long nitems = ctr[kBN + k % 3];
     unsigned long long *dcount = &ctr[kD + (k + 1) % 3];
     if (PROF && blockIdx.x == 0 && threadIdx.x == 0 && (int64_t)k < nk_cap) {
-        rstat[8 * k + 1] = (int64_t)ctr[kI + k % 3];
-        rstat[8 * k + 2] = (int64_t)ctr[kBE + k % 3];
-        rstat[8 * k + 3] = (int64_t)nitems;
+        rstat[16 * k + 1] = (int64_t)ctr[kI + k % 3];
+        rstat[16 * k + 2] = (int64_t)ctr[kBE + k % 3];
+        rstat[16 * k + 3] = (int64_t)nitems;
     }
     const unsigned lane = lane_id();
     uint32_t nvis = 0;

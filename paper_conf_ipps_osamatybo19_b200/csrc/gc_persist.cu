@@ -207,9 +207,12 @@ __device__ __forceinline__ void stage_append(bool pred, T val, int li, T *buf, i
 // Whole block, at the end of a phase: move the staged entries to the global
 // lists (one atomicAdd per non-empty list) and add the coloured count.
 __device__ __forceinline__ void stage_flush(const Args &a, unsigned long long *cs,
-                                            unsigned long long *dcount, uint32_t *Dout) {
+                                            unsigned long long *dcount, uint32_t *Dout,
+                                            unsigned long long *prof_slot = nullptr,
+                                            unsigned long long phase_t0 = 0) {
     Stage &st = stage();
     __syncthreads();
+    if (prof_slot && threadIdx.x == 0) atomicMax(prof_slot, gtimer() - phase_t0);
     if (threadIdx.x == 0) {
         unsigned long long *ctrs[4] = {&cs[cNQS], &cs[cNQ], dcount, &cs[cWQ]};
         const int caps[4] = {kStNQS, kStNQ, kStD, kStWQ};
@@ -495,13 +498,18 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
             for (int i = 0; i < 8; ++i) cn[i] = 0;
             if (PROF) {
                 a.ctr[kSumD] += N;
-                if ((int64_t)k < a.nk_cap) a.rstat[8 * k] = (int64_t)N;
+                if ((int64_t)k < a.nk_cap) a.rstat[16 * k] = (int64_t)N;
                 t0 = gtimer();
             }
         }
         const uint32_t *Din = a.D[k & 1];
         uint32_t *Dout = a.D[(k + 1) & 1];
         unsigned long long *dcount = &cn[cD];
+        // PROF: longest per-block work time of each phase -> rstat[16k + 8 + phase]
+        unsigned long long tb = PROF ? gtimer() : 0ull;
+        unsigned long long *pslot =
+            (PROF && (int64_t)k < a.nk_cap) ? reinterpret_cast<unsigned long long *>(a.rstat + 16 * k + 8)
+                                            : nullptr;
         const uint32_t thresh = 2u * k;
         // ------------------------------------------------------------ P1
         if (dense || N > 4 * nwarps) {
@@ -538,12 +546,13 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
             for (unsigned long long i = gwarp; i < N; i += nwarps)
                 eval_warp<PROF>(a, cs, Din[i], k, false, nvisE);
         }
-        stage_flush(a, cs, dcount, Dout);
+        stage_flush(a, cs, dcount, Dout, pslot ? pslot + 0 : nullptr, tb);
         if (!phase_barrier(a, 0, k)) return;
+        if (PROF) tb = gtimer();
         if (PROF && gtid == 0) {
             unsigned long long t = gtimer();
             tacc[0] += t - t0;
-            if ((int64_t)k < a.nk_cap) a.rstat[8 * k + 4] = (int64_t)(t - t0);
+            if ((int64_t)k < a.nk_cap) a.rstat[16 * k + 4] = (int64_t)(t - t0);
             t0 = t;
         }
         // ----------------------------------------------------------- P1b
@@ -551,21 +560,23 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
         if (nwq) {
             for (unsigned long long i = gwarp; i < nwq; i += nwarps)
                 eval_warp<PROF>(a, cs, a.WQ[i], k, dense, nvisE);
-            stage_flush(a, cs, dcount, Dout);
+            stage_flush(a, cs, dcount, Dout, pslot ? pslot + 1 : nullptr, tb);
             if (!phase_barrier(a, 1, k)) return;
+            if (PROF) tb = gtimer();
         }
         // ------------------------------------------------------------ P2
         const unsigned long long nsq = cs[cSQ];
         if (nsq) {
             for (unsigned long long i = gwarp; i < nsq; i += nwarps)
                 scan_segment<PROF>(a, cs, a.SQ[i], k, dense, nvisS);
-            stage_flush(a, cs, dcount, Dout);
+            stage_flush(a, cs, dcount, Dout, pslot ? pslot + 2 : nullptr, tb);
             if (!phase_barrier(a, 2, k)) return;
+            if (PROF) tb = gtimer();
         }
         if (PROF && gtid == 0) {
             unsigned long long t = gtimer();
             tacc[1] += t - t0;
-            if ((int64_t)k < a.nk_cap) a.rstat[8 * k + 5] = (int64_t)(t - t0);
+            if ((int64_t)k < a.nk_cap) a.rstat[16 * k + 5] = (int64_t)(t - t0);
             t0 = t;
         }
         // ------------------------------------------------------------ P3
@@ -594,17 +605,17 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
             if (PROF && lane == 0) nvisN += (uint32_t)(re - rs);
         }
         if (PROF && gtid == 0 && (int64_t)k < a.nk_cap) {
-            a.rstat[8 * k + 1] = (int64_t)ncol;
-            a.rstat[8 * k + 2] = (int64_t)cs[cLS];
-            a.rstat[8 * k + 3] = (int64_t)nq;
+            a.rstat[16 * k + 1] = (int64_t)ncol;
+            a.rstat[16 * k + 2] = (int64_t)cs[cLS];
+            a.rstat[16 * k + 3] = (int64_t)nq;
         }
         rem -= ncol;
-        stage_flush(a, cs, dcount, Dout);
+        stage_flush(a, cs, dcount, Dout, pslot ? pslot + 3 : nullptr, tb);
         if (!phase_barrier(a, 3, k)) return;
         if (PROF && gtid == 0) {
             unsigned long long t = gtimer();
             tacc[2] += t - t0;
-            if ((int64_t)k < a.nk_cap) a.rstat[8 * k + 6] = (int64_t)(t - t0);
+            if ((int64_t)k < a.nk_cap) a.rstat[16 * k + 6] = (int64_t)(t - t0);
             t0 = t;
         }
     }

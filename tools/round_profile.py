@@ -34,7 +34,7 @@ def main():
     lu = st.launch_us
     rows = []
     for r in range(R):
-        rs = st.round_stats[8 * r: 8 * r + 8]
+        rs = st.round_stats[16 * r: 16 * r + 16]
         # persistent kernel: per-phase times (ns) are in the round record
         t = [x / 1e3 for x in rs[4:7]] if mode == gcb.MODE_EVENT else lu[per * r: per * r + per]
         rows.append({"k": r, "us": t, "stats": rs})
@@ -46,7 +46,7 @@ def main():
         if not sel:
             continue
         tot = [sum(x["us"][c] for x in sel) for c in range(per)]
-        st4 = [sum(x["stats"][c] for x in sel) for c in range(8)]
+        st4 = [sum(x["stats"][c] for x in sel) for c in range(16)]
         summ.append({"rounds": [lo, min(hi, R)], "us_by_class": tot, "us_total": sum(tot),
                      "stat_sums": st4, "us_per_round": sum(tot) / len(sel)})
     res = {"scale": a.scale, "mode": a.mode, "rounds": R, "n_colors": k, "ms": st.ms,
