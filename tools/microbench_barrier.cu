@@ -44,6 +44,25 @@ __global__ void k_chase(const uint32_t *next, int steps, uint32_t *out, int star
     *out = p;
 }
 
+// every warp chases its own random chain through a big array (loaded GPU)
+__global__ void k_chase_many(const uint32_t *next, size_t n, int steps, uint32_t *out) {
+    const unsigned lane = threadIdx.x & 31;
+    uint32_t p = (uint32_t)(((blockIdx.x * blockDim.x + threadIdx.x) >> 5) * 2654435761u % n);
+    if (lane == 0)
+        for (int i = 0; i < steps; ++i) p = next[p];
+    if (lane == 0 && p == 0xFFFFFFFFu) *out = p;
+}
+
+// cost of __threadfence with outstanding stores
+__global__ void k_fence(uint32_t *buf, int iters, unsigned long long *cyc) {
+    unsigned long long t0 = clock64();
+    for (int i = 0; i < iters; ++i) {
+        buf[(threadIdx.x + i * 977) & 0xFFFFF] = i;
+        __threadfence();
+    }
+    if (threadIdx.x == 0) cyc[blockIdx.x] = clock64() - t0;
+}
+
 int main() {
     int sms = 0;
     cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, 0);
@@ -108,6 +127,47 @@ int main() {
                1e6 * ms / steps);
         cudaFree(d);
         cudaFree(o);
+    }
+    {
+        size_t n = (size_t)1 << 29;  // 2 GiB of uint32
+        uint32_t *d, *o;
+        cudaMalloc(&d, n * 4);
+        cudaMalloc(&o, 4);
+        // next[i] = hash(i) mod n: a random functional graph (good enough)
+        std::vector<uint32_t> h(1 << 20);
+        for (size_t c = 0; c < n; c += h.size()) {
+            for (size_t i = 0; i < h.size(); ++i) {
+                uint64_t x = (c + i) * 0x9E3779B97F4A7C15ull;
+                x ^= x >> 29; x *= 0xBF58476D1CE4E5B9ull; x ^= x >> 32;
+                h[i] = (uint32_t)(x % n);
+            }
+            cudaMemcpy(d + c, h.data(), h.size() * 4, cudaMemcpyHostToDevice);
+        }
+        int sms = 0;
+        cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, 0);
+        for (int warps_per_sm : {1, 8, 32}) {
+            int steps = 2000;
+            k_chase_many<<<sms, 32 * warps_per_sm>>>(d, n, 100, o);
+            cudaEventRecord(a);
+            k_chase_many<<<sms, 32 * warps_per_sm>>>(d, n, steps, o);
+            cudaEventRecord(b);
+            cudaEventSynchronize(b);
+            float ms;
+            cudaEventElapsedTime(&ms, a, b);
+            printf("loaded chase, 2 GiB, %d warps/SM (%d warps): %.1f ns per dependent load\n",
+                   warps_per_sm, warps_per_sm * sms, 1e6 * ms / steps);
+        }
+        unsigned long long *cyc;
+        cudaMalloc(&cyc, sizeof(unsigned long long) * sms);
+        k_fence<<<sms, 32>>>(d, 1000, cyc);
+        cudaEventRecord(a);
+        k_fence<<<sms, 32>>>(d, 1000, cyc);
+        cudaEventRecord(b);
+        cudaEventSynchronize(b);
+        float ms;
+        cudaEventElapsedTime(&ms, a, b);
+        printf("store + __threadfence: %.1f ns per iteration (1 warp/SM)\n", 1e6 * ms / 1000);
+        cudaFree(d);
     }
     return 0;
 }
