@@ -258,6 +258,51 @@ __device__ __forceinline__ void enqueue_notify(const Args &a, unsigned long long
     if (m && lane_id() == (unsigned)(__ffs(m) - 1)) atomicAdd(&st.colored, (unsigned)__popc(m));
 }
 
+// Whole-warp first-hit search of a window [s, lim) of at most kWarpWin
+// entries, issued in one shot: every lane loads its 8 column indices, then
+// the 8 colours, then the hits are resolved in entry order (entry e0 + 32 q +
+// lane) with one ballot per 32-entry row -- two dependent load steps instead
+// of one pair per 64 entries.
+__device__ __forceinline__ void warp_window(const Args &a, uint32_t thresh, uint32_t pv,
+                                            const Resume &r, int64_t s, int64_t lim, Found &f,
+                                            uint32_t &nvis) {
+    constexpr int Q = kWarpWin / 32;
+    const unsigned lane = lane_id();
+    uint32_t u[Q], c[Q];
+#pragma unroll
+    for (int q = 0; q < Q; ++q) {
+        const int64_t e = s + q * 32 + lane;
+        u[q] = e < lim ? a.ci[e] : 0u;
+    }
+#pragma unroll
+    for (int q = 0; q < Q; ++q) {
+        const int64_t e = s + q * 32 + lane;
+        c[q] = e < lim ? a.C[u[q]] : 0u;
+    }
+#pragma unroll
+    for (int q = 0; q < Q; ++q) {
+        const int64_t e = s + q * 32 + lane;
+        nvis += e < lim;
+        bool h = false, l = false;
+        if (e < lim && c[q] >= thresh) {
+            const uint32_t pu = weight_mix(u[q] ^ a.key);
+            h = r.need_hi && e >= r.sh && pu > pv;
+            l = r.need_lo && e >= r.sl && pu < pv;
+        }
+        const unsigned bh = __ballot_sync(kFull, h), bl = __ballot_sync(kFull, l);
+        if (f.hpos < 0 && bh) {
+            const int ln = __ffs(bh) - 1;
+            f.hpos = s + q * 32 + ln;
+            f.hw = __shfl_sync(kFull, u[q], ln);
+        }
+        if (f.lpos < 0 && bl) {
+            const int ln = __ffs(bl) - 1;
+            f.lpos = s + q * 32 + ln;
+            f.lw = __shfl_sync(kFull, u[q], ln);
+        }
+    }
+}
+
 // Whole-warp evaluation of one vertex of D_k (warp-uniform arguments): scan a
 // window; resolved -> settle; otherwise open a long scan (P2).
 template <bool PROF>
@@ -273,8 +318,7 @@ __device__ __forceinline__ void eval_warp(const Args &a, unsigned long long *cs,
     const int64_t lim = min(re, s + (int64_t)kWarpWin);
     Found f;
     uint32_t vis = 0;
-    warp_search(a.ci, a.C, thresh, a.key, weight_mix(v ^ a.key), r.need_hi, r.need_lo, r.sh, r.sl,
-                lim, f, vis);
+    warp_window(a, thresh, weight_mix(v ^ a.key), r, s, lim, f, vis);
     if (PROF) nvis += vis;
     const bool miss_hi = r.need_hi && f.hpos < 0;
     const bool miss_lo = r.need_lo && f.lpos < 0;
@@ -608,6 +652,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
             a.rstat[16 * k + 1] = (int64_t)ncol;
             a.rstat[16 * k + 2] = (int64_t)cs[cLS];
             a.rstat[16 * k + 3] = (int64_t)nq;
+            a.rstat[16 * k + 7] = (int64_t)cs[cSQ];
         }
         rem -= ncol;
         stage_flush(a, cs, dcount, Dout, pslot ? pslot + 3 : nullptr, tb);
