@@ -303,6 +303,13 @@ __device__ __forceinline__ void warp_window(const Args &a, uint32_t thresh, uint
     }
 }
 
+// PROF: longest single operation of a round (SM cycles), rstat[16k + 12 + i]
+__device__ __forceinline__ void prof_max(const Args &a, uint32_t k, int i, long long cycles) {
+    if ((int64_t)k < a.nk_cap && lane_id() == 0)
+        atomicMax(reinterpret_cast<unsigned long long *>(a.rstat + 16 * k + 12 + i),
+                  (unsigned long long)cycles);
+}
+
 // Whole-warp evaluation of one vertex of D_k (warp-uniform arguments): scan a
 // window; resolved -> settle; otherwise open a long scan (P2).
 template <bool PROF>
@@ -432,6 +439,7 @@ __device__ __forceinline__ void scan_segment(const Args &a, unsigned long long *
     }
     last = __shfl_sync(kFull, last, 0);
     if (!last) return;
+    const long long cf0 = PROF ? clock64() : 0;
     // the warp that finished the last segment settles v
     bool colored = false;
     if (lane == 0) {
@@ -455,6 +463,7 @@ __device__ __forceinline__ void scan_segment(const Args &a, unsigned long long *
     }
     colored = __shfl_sync(kFull, colored, 0);
     enqueue_notify(a, cs, colored && lane == 0, v, re - rs, k);
+    if (PROF) prof_max(a, k, 1, clock64() - cf0);
 }
 
 // Lane-serial search of a short window [s, lim) (lim - s <= WIN): all column
@@ -587,8 +596,11 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
                 enqueue_notify(a, cs, colored, v, re - rs, k);
             }
         } else {
-            for (unsigned long long i = gwarp; i < N; i += nwarps)
+            for (unsigned long long i = gwarp; i < N; i += nwarps) {
+                const long long c0 = PROF ? clock64() : 0;
                 eval_warp<PROF>(a, cs, Din[i], k, false, nvisE);
+                if (PROF) prof_max(a, k, 2, clock64() - c0);
+            }
         }
         stage_flush(a, cs, dcount, Dout, pslot ? pslot + 0 : nullptr, tb);
         if (!phase_barrier(a, 0, k)) return;
@@ -611,8 +623,11 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
         // ------------------------------------------------------------ P2
         const unsigned long long nsq = cs[cSQ];
         if (nsq) {
-            for (unsigned long long i = gwarp; i < nsq; i += nwarps)
+            for (unsigned long long i = gwarp; i < nsq; i += nwarps) {
+                const long long c0 = PROF ? clock64() : 0;
                 scan_segment<PROF>(a, cs, a.SQ[i], k, dense, nvisS);
+                if (PROF) prof_max(a, k, 0, clock64() - c0);
+            }
             stage_flush(a, cs, dcount, Dout, pslot ? pslot + 2 : nullptr, tb);
             if (!phase_barrier(a, 2, k)) return;
             if (PROF) tb = gtimer();
@@ -641,12 +656,14 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
         }
         // long rows: one kNotifySeg-entry segment per warp
         for (unsigned long long it = gwarp; it < nq; it += nwarps) {
+            const long long cn0 = PROF ? clock64() : 0;
             const uint2 item = a.NQ[it];
             const uint32_t u = item.x;
             const int64_t rs = a.ro[u] + (int64_t)item.y * kNotifySeg;
             const int64_t re = min(a.ro[u + 1], rs + (int64_t)kNotifySeg);
             notify_entries<kNotifySeg / 32>(a, u, rs + lane, re, 32, k, Dout, dcount);
             if (PROF && lane == 0) nvisN += (uint32_t)(re - rs);
+            if (PROF) prof_max(a, k, 3, clock64() - cn0);
         }
         if (PROF && gtid == 0 && (int64_t)k < a.nk_cap) {
             a.rstat[16 * k + 1] = (int64_t)ncol;
