@@ -268,6 +268,7 @@ int ensure_scratch(gc_graph *g, bool need_event, bool need_luby) {
         GC_CUDA_TRY(cudaMalloc(&s.Q2, (nn + (size_t)g->nnz / 128 + 1) * 8));
         GC_CUDA_TRY(cudaMalloc(&s.Q3, (nn + (size_t)g->nnz / 128 + 1) * 8));
         GC_CUDA_TRY(cudaMalloc(&s.LS, nn * 32));
+        GC_CUDA_TRY(cudaMalloc(&s.M, ((nn + 31) / 32) * 4));
     }
     return GC_OK;
 }
@@ -335,6 +336,7 @@ static void free_scratch(Scratch &s) {
     cudaFree(s.Q2);
     cudaFree(s.Q3);
     cudaFree(s.LS);
+    cudaFree(s.M);
     cudaFree(s.ctr);
     cudaFree(s.nk);
     cudaFree(s.rstat);

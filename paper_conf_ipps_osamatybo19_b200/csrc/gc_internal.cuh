@@ -49,6 +49,7 @@ struct Scratch {
     uint32_t *Q2 = nullptr;       // event mode: long-row notify / long-scan segment queue
     uint32_t *Q3 = nullptr;       // persistent event mode: notify segment queue
     void *LS = nullptr;           // persistent event mode: long-scan slots (32 B each)
+    uint32_t *M = nullptr;        // persistent event mode: round-start status bitmask
     uint32_t *S = nullptr;        // Luby inner-loop state / event stamps
     uint32_t *W = nullptr;        // event mode: witness pairs (2 per vertex)
     uint32_t *P = nullptr;        // event mode: resume cursors (2 per vertex)

@@ -70,6 +70,7 @@ struct Args {
     uint2 *W;
     uint2 *P;
     uint32_t *S;
+    uint32_t *M;     // bit u set iff u was uncoloured at the start of this round
     uint32_t *D[2];
     uint32_t *WQ;
     uint2 *SQ;
@@ -97,6 +98,31 @@ __device__ __forceinline__ void flag_error(const Args &a, unsigned kind, uint32_
         a.ctr[kErr + 2] = v;
     }
     a.ctr[kErrPar + (k & 1)] = 1;
+}
+
+// Round-start status (the snapshot of Alg.5 L26, R6) as a 2 MB-per-16M-vertex
+// bitmask that stays in L2: bits are cleared in P3 for the vertices coloured
+// in the round, so the scans of P1 / P2 read exactly the round-start state and
+// colours written concurrently in the round still count as uncoloured.
+__device__ __forceinline__ bool active(const Args &a, uint32_t u) {
+    return (a.M[u >> 5] >> (u & 31)) & 1u;
+}
+
+// Where a vertex resumes (cf. gc_event_common resume_of, with the bitmask).
+__device__ __forceinline__ Resume resume_m(const Args &a, uint32_t v, int64_t rs, bool dense) {
+    Resume r;
+    if (dense) {
+        r.need_hi = r.need_lo = true;
+        r.sh = r.sl = rs;
+    } else {
+        const uint2 w = a.W[v];
+        const uint2 p = a.P[v];
+        r.need_hi = !active(a, w.x);  // hi witness coloured in an earlier round
+        r.need_lo = !active(a, w.y);
+        r.sh = rs + (int64_t)p.x + 1;
+        r.sl = rs + (int64_t)p.y + 1;
+    }
+    return r;
 }
 
 __device__ __forceinline__ unsigned long long gtimer() {
@@ -277,14 +303,14 @@ __device__ __forceinline__ void warp_window(const Args &a, uint32_t thresh, uint
 #pragma unroll
     for (int q = 0; q < Q; ++q) {
         const int64_t e = s + q * 32 + lane;
-        c[q] = e < lim ? a.C[u[q]] : 0u;
+        c[q] = e < lim ? (uint32_t)active(a, u[q]) : 0u;
     }
 #pragma unroll
     for (int q = 0; q < Q; ++q) {
         const int64_t e = s + q * 32 + lane;
         nvis += e < lim;
         bool h = false, l = false;
-        if (e < lim && c[q] >= thresh) {
+        if (e < lim && c[q]) {
             const uint32_t pu = weight_mix(u[q] ^ a.key);
             h = r.need_hi && e >= r.sh && pu > pv;
             l = r.need_lo && e >= r.sl && pu < pv;
@@ -318,7 +344,7 @@ __device__ __forceinline__ void eval_warp(const Args &a, unsigned long long *cs,
     const uint32_t thresh = 2u * k;
     const unsigned lane = lane_id();
     const int64_t rs = a.ro[v], re = a.ro[v + 1];
-    const Resume r = resume_of(v, rs, dense, a.W, a.P, a.C, thresh);
+    const Resume r = resume_m(a, v, rs, dense);
     if (!r.need_hi && !r.need_lo) return;
     int64_t s = r.need_hi ? r.sh : re;
     if (r.need_lo && r.sl < s) s = r.sl;
@@ -408,13 +434,13 @@ __device__ __forceinline__ void scan_segment(const Args &a, unsigned long long *
 #pragma unroll
         for (int q = 0; q < kSeg / 32; ++q) {
             const int64_t e = e0 + q * 32 + lane;
-            c[q] = e < e1 ? a.C[u[q]] : 0u;
+            c[q] = e < e1 ? (uint32_t)active(a, u[q]) : 0u;
         }
         uint32_t rh = kNone, rl = kNone;
 #pragma unroll
         for (int q = 0; q < kSeg / 32; ++q) {
             const int64_t e = e0 + q * 32 + lane;
-            if (e < e1 && c[q] >= thresh) {
+            if (e < e1 && c[q]) {
                 const uint32_t pu = weight_mix(u[q] ^ a.key);
                 const uint32_t rel = (uint32_t)(e - rs);
                 if (want_hi && rel >= L->sh && pu > pv) rh = min(rh, rel);
@@ -448,7 +474,7 @@ __device__ __forceinline__ void scan_segment(const Args &a, unsigned long long *
         const bool bad = (mH != kNone && mH >= (uint32_t)(re - rs)) ||
                          (mL != kNone && mL >= (uint32_t)(re - rs));
         if (bad) flag_error(a, 13 + (mH != kNone && mH >= (uint32_t)(re - rs) ? 0 : 1), k, v);
-        const Resume r = resume_of(v, rs, dense, a.W, a.P, a.C, thresh);
+        const Resume r = resume_m(a, v, rs, dense);
         Found f;
         if (mH != kNone && !bad) {
             f.hpos = rs + mH;
@@ -476,11 +502,11 @@ __device__ __forceinline__ void lane_window(const Args &a, uint32_t thresh, uint
 #pragma unroll
     for (int q = 0; q < WIN; ++q) u[q] = s + q < lim ? a.ci[s + q] : 0u;
 #pragma unroll
-    for (int q = 0; q < WIN; ++q) c[q] = s + q < lim ? a.C[u[q]] : 0u;
+    for (int q = 0; q < WIN; ++q) c[q] = s + q < lim ? (uint32_t)active(a, u[q]) : 0u;
 #pragma unroll
     for (int q = 0; q < WIN; ++q) {
         const int64_t e = s + q;
-        if (e < lim && c[q] >= thresh) {
+        if (e < lim && c[q]) {
             const uint32_t pu = weight_mix(u[q] ^ a.key);
             if (r.need_hi && f.hpos < 0 && e >= r.sh && pu > pv) {
                 f.hpos = e;
@@ -576,7 +602,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
                     v = dense ? (uint32_t)idx : Din[idx];
                     rs = a.ro[v];
                     re = a.ro[v + 1];
-                    r = resume_of(v, rs, dense, a.W, a.P, a.C, thresh);
+                    r = resume_m(a, v, rs, dense);
                 }
                 const bool work = valid && (r.need_hi || r.need_lo);
                 int64_t s = r.need_hi ? r.sh : re;
@@ -650,6 +676,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
                 u = a.NQS[idx];
                 rs = a.ro[u];
                 re = a.ro[u + 1];
+                if ((lane & 7) == 0) atomicAnd(&a.M[u >> 5], ~(1u << (u & 31)));  // coloured now
             }
             notify_entries<4>(a, u, rs + (lane & 7), re, 8, k, Dout, dcount);
             if (PROF && (lane & 7) == 0) nvisN += (uint32_t)(re - rs);
@@ -659,6 +686,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
             const long long cn0 = PROF ? clock64() : 0;
             const uint2 item = a.NQ[it];
             const uint32_t u = item.x;
+            if (item.y == 0 && lane == 0) atomicAnd(&a.M[u >> 5], ~(1u << (u & 31)));
             const int64_t rs = a.ro[u] + (int64_t)item.y * kNotifySeg;
             const int64_t re = min(a.ro[u + 1], rs + (int64_t)kNotifySeg);
             notify_entries<kNotifySeg / 32>(a, u, rs + lane, re, 32, k, Dout, dcount);
@@ -728,6 +756,7 @@ int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     int rc = fill_u32(s.C, GC_UNC, n, g->stream);  // Alg.5 L5
     if (rc) return rc;
     GC_CUDA_TRY(cudaMemsetAsync(s.S, 0, sizeof(uint32_t) * (size_t)n, g->stream));
+    GC_CUDA_TRY(cudaMemsetAsync(s.M, 0xFF, sizeof(uint32_t) * (size_t)((n + 31) / 32), g->stream));
     GC_CUDA_TRY(cudaMemsetAsync(s.ctr, 0, 64 * sizeof(unsigned long long), g->stream));
     const unsigned long long rem = (unsigned long long)n;
     GC_CUDA_TRY(cudaMemcpyAsync(s.ctr + kRem, &rem, sizeof(rem), cudaMemcpyHostToDevice, g->stream));
@@ -744,6 +773,7 @@ int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     a.W = reinterpret_cast<uint2 *>(s.W);
     a.P = reinterpret_cast<uint2 *>(s.P);
     a.S = s.S;
+    a.M = s.M;
     a.D[0] = s.F[0];
     a.D[1] = s.F[1];
     a.WQ = s.hub;
