@@ -87,7 +87,8 @@ typedef enum gc_status {
                                       little overhead, so keep it out of timed runs) */
 
 /* Sweep strategy (gc_options.mode).  All modes return identical colours. */
-#define GC_MODE_AUTO 0   /* EVENT for max-min/multi-hash, SWEEP for Luby */
+#define GC_MODE_AUTO 0   /* max-min: SWEEP if max degree <= 32, else EVENT;
+                            multi-hash and Luby: SWEEP */
 #define GC_MODE_SWEEP 1  /* every round re-scans each uncoloured vertex's row
                             with early exit (the paper's ComputeOp shape) */
 #define GC_MODE_EVENT 2  /* work-efficient: per-vertex witnesses + resume

@@ -519,7 +519,11 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
 
     const bool luby = kind == GC_LUBY_MIS;
     int mode = o->mode;
-    if (mode == GC_MODE_AUTO) mode = GC_MODE_EVENT;
+    // AUTO: on low-degree graphs (meshes, grids) a colouring takes few rounds
+    // and the plain sweep is fastest (measured: 128^3 mesh 0.47 ms sweep vs
+    // 0.77 ms event); skewed graphs take thousands of rounds and need the
+    // work-efficient event mode (R-MAT s24: 107 ms event vs 1689 ms sweep).
+    if (mode == GC_MODE_AUTO) mode = g->max_deg <= 32 ? GC_MODE_SWEEP : GC_MODE_EVENT;
     if (luby) mode = GC_MODE_SWEEP;
     if (mode != GC_MODE_SWEEP && H != 1) mode = GC_MODE_SWEEP;
 
