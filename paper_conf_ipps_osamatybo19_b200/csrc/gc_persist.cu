@@ -146,6 +146,21 @@ __device__ __forceinline__ unsigned long long ld_acquire(const unsigned long lon
     return v;
 }
 
+// release-ordered arrival (MEMBAR.ALL.GPU + atomic; a __threadfence is the
+// much slower sequentially consistent MEMBAR.SC.GPU) and acquire-ordered
+// loads (which also invalidate this SM's L1: CCTL.IVALL)
+__device__ __forceinline__ unsigned long long atom_add_release(unsigned long long *p,
+                                                               unsigned long long x) {
+    unsigned long long v;
+    asm volatile("atom.add.release.gpu.global.u64 %0, [%1], %2;" : "=l"(v) : "l"(p), "l"(x) : "memory");
+    return v;
+}
+__device__ __forceinline__ uint32_t atom_sub_acq_rel(uint32_t *p, uint32_t x) {
+    uint32_t v;
+    asm volatile("atom.add.acq_rel.gpu.global.u32 %0, [%1], %2;" : "=r"(v) : "l"(p), "r"(0u - x) : "memory");
+    return v;
+}
+
 __device__ __forceinline__ bool phase_barrier(const Args &a, int id, uint32_t k) {
     __shared__ int ok_sh;
     __syncthreads();
@@ -153,8 +168,7 @@ __device__ __forceinline__ bool phase_barrier(const Args &a, int id, uint32_t k)
         // monotone arrival counter: barrier instance i completes when it
         // reaches (i + 1) * gridDim.x -- one atomic per block, no reset
         int ok = 1;
-        __threadfence();
-        const unsigned long long old = atomicAdd(a.ctr + kBar, 1ull);
+        const unsigned long long old = atom_add_release(a.ctr + kBar, 1ull);
         const unsigned long long target = (old / gridDim.x + 1) * gridDim.x;
         unsigned spins = 0;
         const unsigned long long t0 = gtimer();
@@ -172,8 +186,7 @@ __device__ __forceinline__ bool phase_barrier(const Args &a, int id, uint32_t k)
                 }
             }
         }
-        __threadfence();  // gpu-scope fence after the wait: also invalidates this SM's L1
-        ok_sh = ok;
+        ok_sh = ok;  // the acquire loads of the spin invalidated this SM's L1
     }
     __syncthreads();
     return ok_sh != 0;
@@ -459,17 +472,13 @@ __device__ __forceinline__ void scan_segment(const Args &a, unsigned long long *
         }
     }
     bool last = false;
-    if (lane == 0) {
-        __threadfence();
-        last = atomicSub(&L->ticket, 1u) == 1u;
-    }
+    if (lane == 0) last = atom_sub_acq_rel(&L->ticket, 1u) == 1u;
     last = __shfl_sync(kFull, last, 0);
     if (!last) return;
     const long long cf0 = PROF ? clock64() : 0;
     // the warp that finished the last segment settles v
     bool colored = false;
     if (lane == 0) {
-        __threadfence();
         const uint32_t mH = atomicAdd(&L->minH, 0u), mL = atomicAdd(&L->minL, 0u);
         const bool bad = (mH != kNone && mH >= (uint32_t)(re - rs)) ||
                          (mL != kNone && mL >= (uint32_t)(re - rs));

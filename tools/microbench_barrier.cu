@@ -32,6 +32,46 @@ __global__ void k_mybar(unsigned long long *ctr, int iters) {
     for (int i = 0; i < iters; ++i) my_barrier(ctr);
 }
 
+// the kernel's barrier: monotone counter, fence + relaxed atomic, acquire
+// spin, trailing fence
+__device__ __forceinline__ unsigned long long ld_acq(const unsigned long long *p) {
+    unsigned long long v;
+    asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+    return v;
+}
+__device__ __forceinline__ unsigned long long atom_add_rel(unsigned long long *p, unsigned long long x) {
+    unsigned long long v;
+    asm volatile("atom.add.release.gpu.global.u64 %0, [%1], %2;" : "=l"(v) : "l"(p), "l"(x) : "memory");
+    return v;
+}
+__global__ void k_monobar(unsigned long long *ctr, int iters) {
+    for (int i = 0; i < iters; ++i) {
+        __syncthreads();
+        if (threadIdx.x == 0) {
+            __threadfence();
+            const unsigned long long old = atomicAdd(ctr, 1ull);
+            const unsigned long long target = (old / gridDim.x + 1) * gridDim.x;
+            while (ld_acq(ctr) < target) {
+            }
+            __threadfence();
+        }
+        __syncthreads();
+    }
+}
+// release-atomic arrival, acquire spin, no explicit fences
+__global__ void k_relbar(unsigned long long *ctr, int iters) {
+    for (int i = 0; i < iters; ++i) {
+        __syncthreads();
+        if (threadIdx.x == 0) {
+            const unsigned long long old = atom_add_rel(ctr, 1ull);
+            const unsigned long long target = (old / gridDim.x + 1) * gridDim.x;
+            while (ld_acq(ctr) < target) {
+            }
+        }
+        __syncthreads();
+    }
+}
+
 __global__ void k_cgbar(int iters) {
     cg::grid_group g = cg::this_grid();
     for (int i = 0; i < iters; ++i) g.sync();
@@ -94,8 +134,24 @@ int main() {
             cudaEventSynchronize(b);
             float ms2;
             cudaEventElapsedTime(&ms2, a, b);
-            printf("barrier: %d blocks x %d threads: mine %.3f us, cg %.3f us  (%s)\n", blocks,
-                   threads, 1e3 * ms / iters, 1e3 * ms2 / iters,
+            float ms3, ms4;
+            cudaMemset(ctr, 0, 64);
+            cudaLaunchCooperativeKernel((void *)k_monobar, blocks, threads, args, 0, 0);
+            cudaEventRecord(a);
+            cudaLaunchCooperativeKernel((void *)k_monobar, blocks, threads, args, 0, 0);
+            cudaEventRecord(b);
+            cudaEventSynchronize(b);
+            cudaEventElapsedTime(&ms3, a, b);
+            cudaMemset(ctr, 0, 64);
+            cudaLaunchCooperativeKernel((void *)k_relbar, blocks, threads, args, 0, 0);
+            cudaEventRecord(a);
+            cudaLaunchCooperativeKernel((void *)k_relbar, blocks, threads, args, 0, 0);
+            cudaEventRecord(b);
+            cudaEventSynchronize(b);
+            cudaEventElapsedTime(&ms4, a, b);
+            printf("barrier: %d blocks x %d threads: gen %.3f us, mono+fences %.3f us, "
+                   "release/acquire %.3f us, cg %.3f us  (%s)\n", blocks, threads,
+                   1e3 * ms / iters, 1e3 * ms3 / iters, 1e3 * ms4 / iters, 1e3 * ms2 / iters,
                    cudaGetErrorString(cudaGetLastError()));
         }
     }
