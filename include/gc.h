@@ -186,6 +186,13 @@ int64_t gc_count_colors(const int32_t *colors, int64_t n);
 /* Library build information (e.g. "gc 1 sm_100a cuda 12.9"). */
 const char *gc_version(void);
 
+/* Memory: device and pinned-host blocks released by gc_destroy are kept in a
+ * per-device cache and reused by later handles (creating a handle then maps
+ * no new pages; a cudaMalloc that fails first returns the cache to the
+ * driver).  gc_trim returns every cached block to the driver now; GC_OK.
+ * Setting GC_NO_CACHE=1 in the environment disables the cache. */
+int gc_trim(void);
+
 /* ---------------------------------------------------- distributed (1D) */
 /* Create a rank's share of a graph partitioned by contiguous vertex ranges:
  * this rank owns rows [v_begin, v_end) of an n_global-vertex graph.

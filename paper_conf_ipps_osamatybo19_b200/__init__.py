@@ -40,7 +40,7 @@ MODE_AUTO, MODE_SWEEP, MODE_EVENT, MODE_EVENT_MULTI = 0, 1, 2, 3
 
 EXPORTS = ["gc_create_csr", "gc_color", "gc_color_ex", "gc_set_stream", "gc_destroy",
            "gc_last_error", "gc_priorities", "gc_count_colors", "gc_version",
-           "gc_create_csr_dist", "gc_nccl_unique_id", "gc_create_csr_loopback"]
+           "gc_trim", "gc_create_csr_dist", "gc_nccl_unique_id", "gc_create_csr_loopback"]
 
 
 class GCError(RuntimeError):
@@ -94,6 +94,7 @@ def lib():
         L.gc_priorities.argtypes, L.gc_priorities.restype = [u64, i32, i64, i64, P], ctypes.c_int
         L.gc_count_colors.argtypes, L.gc_count_colors.restype = [P, i64], i64
         L.gc_version.argtypes, L.gc_version.restype = [], ctypes.c_char_p
+        L.gc_trim.argtypes, L.gc_trim.restype = [], ctypes.c_int
         L.gc_create_csr_dist.argtypes = [i64, i64, i64, i64, P, P, P, ctypes.c_int, ctypes.c_int,
                                          u32, ctypes.POINTER(P)]
         L.gc_create_csr_dist.restype = ctypes.c_int
@@ -280,3 +281,8 @@ def count_colors(colors) -> int:
 
 def version() -> str:
     return lib().gc_version().decode()
+
+
+def trim() -> None:
+    """Return the library's cached device / pinned blocks to the driver."""
+    _check(lib().gc_trim())

@@ -227,8 +227,8 @@ int ensure_nk(gc_graph *g, int64_t need) {
     if (need <= s.nk_cap) return GC_OK;
     int64_t cap = std::max<int64_t>(need * 2, 1 << 12);
     int64_t *nk = nullptr, *rstat = nullptr;
-    GC_CUDA_TRY(cudaMalloc(&nk, sizeof(int64_t) * cap));
-    GC_CUDA_TRY(cudaMalloc(&rstat, sizeof(int64_t) * 16 * cap));
+    GC_CUDA_TRY(dmalloc(&nk, sizeof(int64_t) * cap));
+    GC_CUDA_TRY(dmalloc(&rstat, sizeof(int64_t) * 16 * cap));
     GC_CUDA_TRY(cudaMemsetAsync(rstat, 0, sizeof(int64_t) * 16 * cap, g->stream));
     if (s.nk) {
         GC_CUDA_TRY(cudaMemcpyAsync(nk, s.nk, sizeof(int64_t) * s.nk_cap, cudaMemcpyDeviceToDevice,
@@ -236,8 +236,8 @@ int ensure_nk(gc_graph *g, int64_t need) {
         GC_CUDA_TRY(cudaMemcpyAsync(rstat, s.rstat, sizeof(int64_t) * 16 * s.nk_cap,
                                     cudaMemcpyDeviceToDevice, g->stream));
         GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
-        cudaFree(s.nk);
-        cudaFree(s.rstat);
+        dfree(s.nk);
+        dfree(s.rstat);
     }
     s.nk = nk;
     s.rstat = rstat;
@@ -249,26 +249,26 @@ int ensure_scratch(gc_graph *g, bool need_event, bool need_luby) {
     Scratch &s = g->s;
     const size_t nn = (size_t)std::max<int64_t>(g->n, 1);
     if (!s.C) {
-        GC_CUDA_TRY(cudaMalloc(&s.C, nn * 4));
-        GC_CUDA_TRY(cudaMalloc(&s.F[0], nn * 4));
-        GC_CUDA_TRY(cudaMalloc(&s.F[1], nn * 4));
-        GC_CUDA_TRY(cudaMalloc(&s.hub, nn * 4));
-        GC_CUDA_TRY(cudaMalloc(&s.ctr, kCtrWords * sizeof(unsigned long long)));
+        GC_CUDA_TRY(dmalloc(&s.C, nn * 4));
+        GC_CUDA_TRY(dmalloc(&s.F[0], nn * 4));
+        GC_CUDA_TRY(dmalloc(&s.F[1], nn * 4));
+        GC_CUDA_TRY(dmalloc(&s.hub, nn * 4));
+        GC_CUDA_TRY(dmalloc(&s.ctr, kCtrWords * sizeof(unsigned long long)));
         GC_CUDA_TRY(cudaMemset(s.ctr, 0, kCtrWords * sizeof(unsigned long long)));
-        GC_CUDA_TRY(cudaMallocHost(&s.host_pinned, 4096));
+        GC_CUDA_TRY(hmalloc(&s.host_pinned, 4096));
         int rc = ensure_nk(g, 1 << 12);
         if (rc) return rc;
     }
-    if ((need_luby || need_event) && !s.S) GC_CUDA_TRY(cudaMalloc(&s.S, nn * 4));
+    if ((need_luby || need_event) && !s.S) GC_CUDA_TRY(dmalloc(&s.S, nn * 4));
     if (need_event && !s.W) {
-        GC_CUDA_TRY(cudaMalloc(&s.W, nn * 8));
-        GC_CUDA_TRY(cudaMalloc(&s.P, nn * 8));
-        GC_CUDA_TRY(cudaMalloc(&s.Q, nn * 4));
+        GC_CUDA_TRY(dmalloc(&s.W, nn * 8));
+        GC_CUDA_TRY(dmalloc(&s.P, nn * 8));
+        GC_CUDA_TRY(dmalloc(&s.Q, nn * 4));
         // long-row notify items (u, segment): at most n + nnz/128 per round
-        GC_CUDA_TRY(cudaMalloc(&s.Q2, (nn + (size_t)g->nnz / 128 + 1) * 8));
-        GC_CUDA_TRY(cudaMalloc(&s.Q3, (nn + (size_t)g->nnz / 128 + 1) * 8));
-        GC_CUDA_TRY(cudaMalloc(&s.LS, nn * 32));
-        GC_CUDA_TRY(cudaMalloc(&s.M, ((nn + 31) / 32) * 4));
+        GC_CUDA_TRY(dmalloc(&s.Q2, (nn + (size_t)g->nnz / 128 + 1) * 8));
+        GC_CUDA_TRY(dmalloc(&s.Q3, (nn + (size_t)g->nnz / 128 + 1) * 8));
+        GC_CUDA_TRY(dmalloc(&s.LS, nn * 32));
+        GC_CUDA_TRY(dmalloc(&s.M, ((nn + 31) / 32) * 4));
     }
     return GC_OK;
 }
@@ -293,9 +293,9 @@ int64_t count_colors_device(gc_graph *g, const uint32_t *C, int64_t n, bool comp
     }
     const int64_t words = (int64_t)(maxc >> 5) + 1;
     if (words > s.bitmap_words) {
-        if (s.bitmap) cudaFree(s.bitmap);
+        if (s.bitmap) dfree(s.bitmap);
         s.bitmap = nullptr;
-        GC_CUDA_TRY(cudaMalloc(&s.bitmap, (size_t)words * 8));  // bitmap + rank table
+        GC_CUDA_TRY(dmalloc(&s.bitmap, (size_t)words * 8));  // bitmap + rank table
         s.bitmap_words = words;
     }
     uint32_t *rank = s.bitmap + words;
@@ -325,23 +325,24 @@ int launch_priorities(uint64_t seed, int j, int64_t v_begin, int64_t count, uint
 }
 
 static void free_scratch(Scratch &s) {
-    cudaFree(s.C);
-    cudaFree(s.F[0]);
-    cudaFree(s.F[1]);
-    cudaFree(s.hub);
-    cudaFree(s.S);
-    cudaFree(s.W);
-    cudaFree(s.P);
-    cudaFree(s.Q);
-    cudaFree(s.Q2);
-    cudaFree(s.Q3);
-    cudaFree(s.LS);
-    cudaFree(s.M);
-    cudaFree(s.ctr);
-    cudaFree(s.nk);
-    cudaFree(s.rstat);
-    cudaFree(s.bitmap);
-    if (s.host_pinned) cudaFreeHost(s.host_pinned);
+    dfree(s.C);
+    dfree(s.F[0]);
+    dfree(s.F[1]);
+    dfree(s.hub);
+    dfree(s.S);
+    dfree(s.W);
+    dfree(s.P);
+    dfree(s.Q);
+    dfree(s.Q2);
+    dfree(s.Q3);
+    dfree(s.LS);
+    dfree(s.M);
+    dfree(s.ctr);
+    dfree(s.nk);
+    dfree(s.rstat);
+    dfree(s.bitmap);
+    dfree(s.hist);
+    if (s.host_pinned) hfree(s.host_pinned);
     s = Scratch();
 }
 
@@ -392,8 +393,8 @@ int gc_create_csr_internal(int64_t n, int64_t nnz, const int64_t *row_offsets,
     const bool ci_dev = nnz == 0 || is_device_ptr(col_indices);
     auto fail = [&](int code) {
         if (g->owns_csr) {
-            cudaFree(g->ro);
-            cudaFree(g->ci);
+            dfree(g->ro);
+            dfree(g->ci);
         }
         free_scratch(g->s);
         delete g;
@@ -404,9 +405,9 @@ int gc_create_csr_internal(int64_t n, int64_t nnz, const int64_t *row_offsets,
         g->ro = const_cast<int64_t *>(row_offsets);
         g->ci = const_cast<uint32_t *>(col_indices);
     } else {
-        cudaError_t e = cudaMalloc(&g->ro, sizeof(int64_t) * (size_t)(n + 1));
-        if (e == cudaSuccess) e = cudaMalloc(&g->ci, sizeof(uint32_t) * (size_t)std::max<int64_t>(nnz, 1));
-        if (e != cudaSuccess) return fail(cuda_fail(e, "cudaMalloc(csr)"));
+        cudaError_t e = dmalloc(&g->ro, sizeof(int64_t) * (size_t)(n + 1));
+        if (e == cudaSuccess) e = dmalloc(&g->ci, sizeof(uint32_t) * (size_t)std::max<int64_t>(nnz, 1));
+        if (e != cudaSuccess) return fail(cuda_fail(e, "dmalloc(csr)"));
         e = cudaMemcpy(g->ro, row_offsets, sizeof(int64_t) * (size_t)(n + 1), cudaMemcpyDefault);
         if (e == cudaSuccess && nnz > 0)
             e = cudaMemcpy(g->ci, col_indices, sizeof(uint32_t) * (size_t)nnz, cudaMemcpyDefault);
@@ -474,10 +475,13 @@ int gc_set_stream(gc_graph *g, void *cuda_stream) {
 void gc_destroy(gc_graph *g) {
     if (!g) return;
     cudaSetDevice(g->device);
+    // blocks go back to the library cache (gc_alloc.cu), so no work that
+    // uses them may still be pending (cudaFree used to imply this sync)
+    cudaDeviceSynchronize();
     destroy_dist(g);
     if (g->owns_csr) {
-        cudaFree(g->ro);
-        cudaFree(g->ci);
+        dfree(g->ro);
+        dfree(g->ci);
     }
     free_scratch(g->s);
     delete g;
@@ -640,13 +644,13 @@ int gc_priorities(uint64_t seed, int32_t j, int64_t v_begin, int64_t count, uint
         return GC_OK;
     }
     uint32_t *d = nullptr;
-    GC_CUDA_TRY(cudaMalloc(&d, sizeof(uint32_t) * (size_t)count));
+    GC_CUDA_TRY(dmalloc(&d, sizeof(uint32_t) * (size_t)count));
     rc = launch_priorities(seed, j, v_begin, count, d, 0);
     if (!rc) {
         cudaError_t e = cudaMemcpy(out, d, sizeof(uint32_t) * (size_t)count, cudaMemcpyDeviceToHost);
         if (e != cudaSuccess) rc = cuda_fail(e, "gc_priorities copy");
     }
-    cudaFree(d);
+    dfree(d);
     return rc;
 }
 
@@ -666,18 +670,18 @@ int64_t gc_count_colors(const int32_t *colors, int64_t n) {
     const uint32_t *C = reinterpret_cast<const uint32_t *>(colors);
     uint32_t *dC = nullptr;
     if (!is_device_ptr(colors)) {
-        GC_CUDA_TRY(cudaMalloc(&dC, sizeof(uint32_t) * (size_t)n));
+        GC_CUDA_TRY(dmalloc(&dC, sizeof(uint32_t) * (size_t)n));
         GC_CUDA_TRY(cudaMemcpy(dC, colors, sizeof(uint32_t) * (size_t)n, cudaMemcpyHostToDevice));
         C = dC;
     }
     int64_t launches = 0;
     int64_t r = GC_OK;
-    cudaError_t e = cudaMalloc(&tmp.s.ctr, kCtrWords * sizeof(unsigned long long));
-    if (e == cudaSuccess) e = cudaMallocHost(&tmp.s.host_pinned, 4096);
+    cudaError_t e = dmalloc(&tmp.s.ctr, kCtrWords * sizeof(unsigned long long));
+    if (e == cudaSuccess) e = hmalloc(&tmp.s.host_pinned, 4096);
     if (e != cudaSuccess) r = cuda_fail(e, "gc_count_colors alloc");
     if (r == GC_OK) r = count_colors_device(&tmp, C, n, false, nullptr, &launches);
     free_scratch(tmp.s);
-    cudaFree(dC);
+    dfree(dC);
     return r;
 }
 

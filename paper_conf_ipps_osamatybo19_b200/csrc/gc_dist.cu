@@ -105,32 +105,32 @@ __global__ void k_rebase(const int64_t *ro, int64_t n_loc, int64_t *out) {
 
 int alloc_part(Part &p, int64_t n_global, int64_t cap, int world) {
     const int64_t nl = std::max<int64_t>(p.v1 - p.v0, 1);
-    GC_CUDA_TRY(cudaMalloc(&p.C, sizeof(uint32_t) * (size_t)std::max<int64_t>(n_global, 1)));
-    GC_CUDA_TRY(cudaMalloc(&p.F[0], sizeof(uint32_t) * (size_t)nl));
-    GC_CUDA_TRY(cudaMalloc(&p.F[1], sizeof(uint32_t) * (size_t)nl));
-    GC_CUDA_TRY(cudaMalloc(&p.hub, sizeof(uint32_t) * (size_t)nl));
-    GC_CUDA_TRY(cudaMalloc(&p.colored, sizeof(uint2) * (size_t)std::max<int64_t>(cap, 1)));
-    GC_CUDA_TRY(cudaMalloc(&p.recv, sizeof(uint2) * (size_t)std::max<int64_t>(cap, 1) * world));
-    GC_CUDA_TRY(cudaMalloc(&p.ctr, 64 * sizeof(unsigned long long)));
-    GC_CUDA_TRY(cudaMalloc(&p.cnt_send, 2 * sizeof(unsigned long long)));
-    GC_CUDA_TRY(cudaMalloc(&p.cnt_recv, 2 * sizeof(unsigned long long) * world));
-    GC_CUDA_TRY(cudaMalloc(&p.nk, sizeof(int64_t)));
+    GC_CUDA_TRY(dmalloc(&p.C, sizeof(uint32_t) * (size_t)std::max<int64_t>(n_global, 1)));
+    GC_CUDA_TRY(dmalloc(&p.F[0], sizeof(uint32_t) * (size_t)nl));
+    GC_CUDA_TRY(dmalloc(&p.F[1], sizeof(uint32_t) * (size_t)nl));
+    GC_CUDA_TRY(dmalloc(&p.hub, sizeof(uint32_t) * (size_t)nl));
+    GC_CUDA_TRY(dmalloc(&p.colored, sizeof(uint2) * (size_t)std::max<int64_t>(cap, 1)));
+    GC_CUDA_TRY(dmalloc(&p.recv, sizeof(uint2) * (size_t)std::max<int64_t>(cap, 1) * world));
+    GC_CUDA_TRY(dmalloc(&p.ctr, 64 * sizeof(unsigned long long)));
+    GC_CUDA_TRY(dmalloc(&p.cnt_send, 2 * sizeof(unsigned long long)));
+    GC_CUDA_TRY(dmalloc(&p.cnt_recv, 2 * sizeof(unsigned long long) * world));
+    GC_CUDA_TRY(dmalloc(&p.nk, sizeof(int64_t)));
     p.nk_cap = 1;
     return GC_OK;
 }
 
 void free_part(Part &p) {
-    if (p.owns_ro) cudaFree(p.ro);
-    cudaFree(p.C);
-    cudaFree(p.F[0]);
-    cudaFree(p.F[1]);
-    cudaFree(p.hub);
-    cudaFree(p.colored);
-    cudaFree(p.recv);
-    cudaFree(p.ctr);
-    cudaFree(p.cnt_send);
-    cudaFree(p.cnt_recv);
-    cudaFree(p.nk);
+    if (p.owns_ro) dfree(p.ro);
+    dfree(p.C);
+    dfree(p.F[0]);
+    dfree(p.F[1]);
+    dfree(p.hub);
+    dfree(p.colored);
+    dfree(p.recv);
+    dfree(p.ctr);
+    dfree(p.cnt_send);
+    dfree(p.cnt_recv);
+    dfree(p.nk);
     p = Part();
 }
 
@@ -161,7 +161,7 @@ void destroy_dist(gc_graph *g) {
     if (!g || !g->dist) return;
     Dist &d = *g->dist;
     for (auto &p : d.parts) free_part(p);
-    if (d.host_cnt) cudaFreeHost(d.host_cnt);
+    if (d.host_cnt) hfree(d.host_cnt);
 #ifdef GC_HAVE_NCCL
     if (d.comm) ncclCommDestroy(d.comm);
 #endif
@@ -317,16 +317,16 @@ int gc_create_csr_dist(int64_t n_global, int64_t v_begin, int64_t v_end, int64_t
     // padding capacity: the largest owned range over all ranks
     unsigned long long *tmp = nullptr;
     unsigned long long mine = (unsigned long long)(v_end - v_begin), mx = 0;
-    cudaError_t ce = cudaMalloc(&tmp, sizeof(unsigned long long));
+    cudaError_t ce = dmalloc(&tmp, sizeof(unsigned long long));
     if (ce == cudaSuccess) ce = cudaMemcpy(tmp, &mine, sizeof(mine), cudaMemcpyHostToDevice);
     if (ce != cudaSuccess) {
-        cudaFree(tmp);
+        dfree(tmp);
         gc_destroy(g);
         return cuda_fail(ce, "dist setup");
     }
     e = ncclAllReduce(tmp, tmp, 1, ncclUint64, ncclMax, d.comm, 0);
     if (e == ncclSuccess) ce = cudaMemcpy(&mx, tmp, sizeof(mx), cudaMemcpyDeviceToHost);
-    cudaFree(tmp);
+    dfree(tmp);
     if (e != ncclSuccess || ce != cudaSuccess) {
         gc_destroy(g);
         return e != ncclSuccess ? nccl_fail(e, "ncclAllReduce") : cuda_fail(ce, "dist setup");
@@ -341,7 +341,7 @@ int gc_create_csr_dist(int64_t n_global, int64_t v_begin, int64_t v_end, int64_t
     p.ci = g->ci;
     p.owns_ro = false;
     rc = alloc_part(p, n_global, d.cap, world);
-    if (rc == GC_OK && cudaMallocHost(&d.host_cnt, 2 * sizeof(unsigned long long) * world) != cudaSuccess)
+    if (rc == GC_OK && hmalloc(&d.host_cnt, 2 * sizeof(unsigned long long) * world) != cudaSuccess)
         rc = GC_ERR_OOM;
     if (rc) {
         gc_destroy(g);
@@ -384,7 +384,7 @@ int gc_create_csr_loopback(int64_t n, int64_t nnz, const int64_t *row_offsets,
         p.v1 = std::min<int64_t>(n, p.v0 + chunk);
         p.nnz = h_ro[p.v1] - h_ro[p.v0];
         p.ci = g->ci + h_ro[p.v0];
-        ce = cudaMalloc(&p.ro, sizeof(int64_t) * (size_t)(p.v1 - p.v0 + 1));
+        ce = dmalloc(&p.ro, sizeof(int64_t) * (size_t)(p.v1 - p.v0 + 1));
         if (ce != cudaSuccess) {
             gc_destroy(g);
             return cuda_fail(ce, "loopback setup");
@@ -397,7 +397,7 @@ int gc_create_csr_loopback(int64_t n, int64_t nnz, const int64_t *row_offsets,
             return rc;
         }
     }
-    if (cudaMallocHost(&d.host_cnt, 2 * sizeof(unsigned long long) * parts) != cudaSuccess) {
+    if (hmalloc(&d.host_cnt, 2 * sizeof(unsigned long long) * parts) != cudaSuccess) {
         gc_destroy(g);
         return GC_ERR_OOM;
     }

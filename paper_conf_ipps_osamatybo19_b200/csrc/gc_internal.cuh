@@ -58,6 +58,7 @@ struct Scratch {
     int64_t nk_cap = 0;
     int64_t *rstat = nullptr;     // PROF: 4 counters per round (cap nk_cap)
     uint32_t *bitmap = nullptr;   // colour-count bitmap
+    unsigned long long *hist = nullptr;  // GC_PROFILE_HIST histograms (gc_persist.cu)
     int64_t bitmap_words = 0;
     int64_t *host_pinned = nullptr;  // pinned readback area
 };
@@ -85,6 +86,21 @@ namespace gc {
 // ----------------------------------------------------------------- errors
 void set_error(const std::string &msg);
 int cuda_fail(cudaError_t e, const char *what);
+
+// gc_alloc.cu: cached device / pinned-host allocations (free only when no
+// pending device work uses the block)
+cudaError_t dmalloc_raw(void **p, size_t bytes);
+void dfree(void *p);
+cudaError_t hmalloc_raw(void **p, size_t bytes);
+void hfree(void *p);
+template <class T>
+inline cudaError_t dmalloc(T **p, size_t bytes) {
+    return dmalloc_raw(reinterpret_cast<void **>(p), bytes);
+}
+template <class T>
+inline cudaError_t hmalloc(T **p, size_t bytes) {
+    return hmalloc_raw(reinterpret_cast<void **>(p), bytes);
+}
 
 #define GC_CUDA_TRY(expr)                                   \
     do {                                                    \

@@ -20,6 +20,7 @@
 // The host launches one kernel per colouring; per-round sizes land in nk[].
 
 #include <cstdio>
+#include <cstdlib>
 
 #include "gc_event_common.cuh"
 
@@ -85,6 +86,7 @@ struct Args {
     uint32_t key;
     uint32_t max_rounds;
     unsigned long long nq_cap, sq_cap, ls_cap;  // queue capacities (items)
+    unsigned long long *hist;  // PROF + GC_PROFILE_HIST: [8][32] log2 histograms, else null
 };
 
 // Internal-consistency trap: record the first violation (kind, round, vertex)
@@ -245,13 +247,26 @@ __device__ __forceinline__ void stage_append(bool pred, T val, int li, T *buf, i
 
 // Whole block, at the end of a phase: move the staged entries to the global
 // lists (one atomicAdd per non-empty list) and add the coloured count.
+// PROF: log2 histogram row `row` of a.hist (rows 0-3: cycles of one segment
+// scan / settle of a long scan / warp evaluation / notify segment; rows 4-7:
+// ns of one block's work in phase P1 / P1b / P2 / P3)
+__device__ __forceinline__ void prof_hist(const Args &a, int row, unsigned long long x) {
+    if (!a.hist) return;
+    const int b = x ? min(31, 63 - __clzll((long long)x)) : 0;
+    atomicAdd(&a.hist[row * 32 + b], 1ull);
+}
+
 __device__ __forceinline__ void stage_flush(const Args &a, unsigned long long *cs,
                                             unsigned long long *dcount, uint32_t *Dout,
                                             unsigned long long *prof_slot = nullptr,
-                                            unsigned long long phase_t0 = 0) {
+                                            unsigned long long phase_t0 = 0, int phase = 0) {
     Stage &st = stage();
     __syncthreads();
-    if (prof_slot && threadIdx.x == 0) atomicMax(prof_slot, gtimer() - phase_t0);
+    if (prof_slot && threadIdx.x == 0) {
+        const unsigned long long dt = gtimer() - phase_t0;
+        atomicMax(prof_slot, dt);
+        prof_hist(a, 4 + phase, dt);
+    }
     if (threadIdx.x == 0) {
         unsigned long long *ctrs[4] = {&cs[cNQS], &cs[cNQ], dcount, &cs[cWQ]};
         const int caps[4] = {kStNQS, kStNQ, kStD, kStWQ};
@@ -347,6 +362,7 @@ __device__ __forceinline__ void prof_max(const Args &a, uint32_t k, int i, long 
     if ((int64_t)k < a.nk_cap && lane_id() == 0)
         atomicMax(reinterpret_cast<unsigned long long *>(a.rstat + 16 * k + 12 + i),
                   (unsigned long long)cycles);
+    if (lane_id() == 0) prof_hist(a, i, (unsigned long long)cycles);
 }
 
 // Whole-warp evaluation of one vertex of D_k (warp-uniform arguments): scan a
@@ -637,7 +653,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
                 if (PROF) prof_max(a, k, 2, clock64() - c0);
             }
         }
-        stage_flush(a, cs, dcount, Dout, pslot ? pslot + 0 : nullptr, tb);
+        stage_flush(a, cs, dcount, Dout, pslot ? pslot + 0 : nullptr, tb, 0);
         if (!phase_barrier(a, 0, k)) return;
         if (PROF) tb = gtimer();
         if (PROF && gtid == 0) {
@@ -651,7 +667,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
         if (nwq) {
             for (unsigned long long i = gwarp; i < nwq; i += nwarps)
                 eval_warp<PROF>(a, cs, a.WQ[i], k, dense, nvisE);
-            stage_flush(a, cs, dcount, Dout, pslot ? pslot + 1 : nullptr, tb);
+            stage_flush(a, cs, dcount, Dout, pslot ? pslot + 1 : nullptr, tb, 1);
             if (!phase_barrier(a, 1, k)) return;
             if (PROF) tb = gtimer();
         }
@@ -663,7 +679,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
                 scan_segment<PROF>(a, cs, a.SQ[i], k, dense, nvisS);
                 if (PROF) prof_max(a, k, 0, clock64() - c0);
             }
-            stage_flush(a, cs, dcount, Dout, pslot ? pslot + 2 : nullptr, tb);
+            stage_flush(a, cs, dcount, Dout, pslot ? pslot + 2 : nullptr, tb, 2);
             if (!phase_barrier(a, 2, k)) return;
             if (PROF) tb = gtimer();
         }
@@ -709,7 +725,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_event_persistent(Args a) {
             a.rstat[16 * k + 7] = (int64_t)cs[cSQ];
         }
         rem -= ncol;
-        stage_flush(a, cs, dcount, Dout, pslot ? pslot + 3 : nullptr, tb);
+        stage_flush(a, cs, dcount, Dout, pslot ? pslot + 3 : nullptr, tb, 3);
         if (!phase_barrier(a, 3, k)) return;
         if (PROF && gtid == 0) {
             unsigned long long t = gtimer();
@@ -800,6 +816,15 @@ int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     a.nq_cap = a.sq_cap = (unsigned long long)(n + g->nnz / 128 + 1);
     a.ls_cap = (unsigned long long)n;
     const bool prof = p.prof && p.prof->on;
+    // GC_PROFILE_HIST=<file>: with GC_PROFILE, append the op-latency
+    // histograms of this colouring to <file> (tools/round_profile.py)
+    const char *hist_path = prof ? std::getenv("GC_PROFILE_HIST") : nullptr;
+    a.hist = nullptr;
+    if (hist_path && hist_path[0]) {
+        if (!s.hist) GC_CUDA_TRY(dmalloc(&s.hist, 8 * 32 * sizeof(unsigned long long)));
+        GC_CUDA_TRY(cudaMemsetAsync(s.hist, 0, 8 * 32 * sizeof(unsigned long long), g->stream));
+        a.hist = s.hist;
+    }
     cudaEvent_t e0 = nullptr, e1 = nullptr;
     if (prof) {
         GC_CUDA_TRY(cudaEventCreate(&e0));
@@ -847,11 +872,23 @@ int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
         // evaluated vertex 4 B (D entry, not in round 0) + 16 B row offsets +
         // 16 B witness state (not in round 0) + 16 B state or 8 B colour/list
         // write; 4 B per scanned entry; per coloured vertex 4 B list + 16 B
-        // offsets; 4 B per notified entry.
+        // offsets; per notified entry 4 B column id + 4 B colour + 8 B witness
+        // ids of the neighbour.
         const int64_t b = 4 * (sumD - n) + 16 * sumD + 16 * (sumD - n) + 16 * (sumD - n) + 8 * n +
-                          4 * (visE + visS) + 20 * n + 4 * visN;
+                          4 * (visE + visS) + 20 * n + 16 * visN;
         p.prof->bytes[0] += b;
         p.prof->visits += visE + visS;
+        if (a.hist) {
+            unsigned long long hh[8 * 32];
+            GC_CUDA_TRY(cudaMemcpy(hh, a.hist, sizeof(hh), cudaMemcpyDeviceToHost));
+            if (FILE *f = std::fopen(hist_path, "a")) {
+                std::fprintf(f, "{\"n\": %lld, \"rounds\": %lld, \"hist\": [", (long long)n,
+                             (long long)r->rounds);
+                for (int i = 0; i < 8 * 32; ++i) std::fprintf(f, "%s%llu", i ? ", " : "", hh[i]);
+                std::fprintf(f, "]}\n");
+                std::fclose(f);
+            }
+        }
     }
     return GC_OK;
 }

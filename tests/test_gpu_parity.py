@@ -208,6 +208,19 @@ def test_borrow_device_and_stream():
         assert (out.cpu().numpy().view(np.uint32) == ref).all()
 
 
+def test_memory_cache_reuse_and_trim():
+    """Handles of different sizes reuse the library's cached blocks (gc_alloc.cu):
+    stale contents of a reused block must never leak into a later colouring."""
+    graphs = [G.rmat(s, 8, seed=s) for s in (13, 11, 13, 12)]
+    refs = [O.color_maxmin(g, 5) for g in graphs]
+    for rep in range(2):
+        for g, ref in zip(graphs, refs):
+            for mode in (gcb.MODE_EVENT, gcb.MODE_SWEEP):
+                got, _, _ = gpu_colors(g, 5, gcb.MAXMIN, mode=mode)
+                assert (got == ref).all()
+        gcb.trim()
+
+
 # ----------------------------------------------------------- config sizes
 @pytest.mark.parametrize("mode", MODES)
 def test_cfg1_grid(mode):

@@ -25,8 +25,12 @@ def main():
     g = G.rmat(a.scale, 16, seed=1, device="cuda")
     mode = {"event": gcb.MODE_EVENT, "sweep": gcb.MODE_SWEEP, "multi": gcb.MODE_EVENT_MULTI}[a.mode]
     out = torch.empty(g.n, dtype=torch.int32, device="cuda")
+    hist_path = a.out + ".hist"
+    if os.path.exists(hist_path):
+        os.remove(hist_path)
     with gcb.Graph(g.n, g.row_offsets, g.col_indices, flags=gcb.BORROW_DEVICE) as h:
         h.color(1, gcb.MAXMIN, out, mode=mode)
+        os.environ["GC_PROFILE_HIST"] = hist_path  # read by libgc at each profiled colouring
         _, k, st = h.color(1, gcb.MAXMIN, out, mode=mode, flags=gcb.PROFILE, stats=True,
                            trace_cap=1 << 15)
     R = st.rounds
@@ -49,8 +53,20 @@ def main():
         st4 = [sum(x["stats"][c] for x in sel) for c in range(16)]
         summ.append({"rounds": [lo, min(hi, R)], "us_by_class": tot, "us_total": sum(tot),
                      "stat_sums": st4, "us_per_round": sum(tot) / len(sel)})
+    hist = None
+    if os.path.exists(hist_path):
+        with open(hist_path) as f:
+            hist = json.loads(f.readlines()[-1])["hist"]
+        names = ["seg scan (cycles)", "long-scan settle (cycles)", "warp eval (cycles)",
+                 "notify segment (cycles)", "block work P1 (ns)", "block work P1b (ns)",
+                 "block work P2 (ns)", "block work P3 (ns)"]
+        hist = {names[i]: {f"2^{b}": hist[32 * i + b] for b in range(32) if hist[32 * i + b]}
+                for i in range(8)}
+        for nm, hh in hist.items():
+            tot = sum(hh.values())
+            print(nm, tot, hh)
     res = {"scale": a.scale, "mode": a.mode, "rounds": R, "n_colors": k, "ms": st.ms,
-           "kernel_ms": st.kernel_ms, "buckets": summ,
+           "kernel_ms": st.kernel_ms, "buckets": summ, "op_histograms": hist,
            "top_rounds": sorted(rows, key=lambda x: -sum(x["us"]))[:25]}
     os.makedirs(os.path.dirname(a.out) or ".", exist_ok=True)
     with open(a.out, "w") as f:
