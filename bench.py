@@ -44,7 +44,7 @@ def parse():
     ap.add_argument("--scale", type=int, default=0, help="R-MAT scale (default 24+log2 N)")
     ap.add_argument("--variant", default="maxmin", choices=["maxmin", "luby", "multihash"])
     ap.add_argument("--hashes", type=int, default=4)
-    ap.add_argument("--mode", default="auto", choices=["auto", "sweep", "event", "event-multi"])
+    ap.add_argument("--mode", default="auto", choices=["auto", "sweep", "event", "event-multi", "count"])
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-profile", action="store_true")
@@ -214,7 +214,7 @@ def main():
     variant = {"maxmin": gcb.MAXMIN, "luby": gcb.LUBY_MIS,
                "multihash": gcb.MULTIHASH(args.hashes)}[args.variant]
     mode = {"auto": gcb.MODE_AUTO, "sweep": gcb.MODE_SWEEP, "event": gcb.MODE_EVENT,
-            "event-multi": gcb.MODE_EVENT_MULTI}[args.mode]
+            "event-multi": gcb.MODE_EVENT_MULTI, "count": gcb.MODE_COUNT}[args.mode]
 
     t0 = time.time()
     if world > 1:
@@ -268,7 +268,8 @@ def main():
         total_ms = float(t.item())
     ms_per = total_ms / args.steps
     value = nnz_global * args.steps / (total_ms / 1e3) / 1e9
-    mode_used = {1: "sweep", 2: "event (persistent)", 3: "event (multi-kernel)"}.get(
+    mode_used = {1: "sweep", 2: "event (persistent)", 3: "event (multi-kernel)",
+                 4: "count (persistent)"}.get(
         st.mode_used, str(st.mode_used))
 
     # ---- roofline of the dominant kernel: a profiled pass (GC_PROFILE brackets
@@ -283,9 +284,11 @@ def main():
                                   2: "phase P1b+P2 long scans", 3: "phase P3 notify"},
                  gcb.MODE_EVENT_MULTI: {0: "k_eval", 1: "k_eval_big", 2: "k_notify",
                                         3: "k_notify_big"},
-                 gcb.MODE_SWEEP: {0: "k_sweep", 1: "k_hub", 2: "other", 3: "other"}}[sp.mode_used]
-        if sp.mode_used == gcb.MODE_EVENT:
-            cls = 0  # one persistent launch; classes 1-3 are its phases (globaltimer)
+                 gcb.MODE_SWEEP: {0: "k_sweep", 1: "k_hub", 2: "other", 3: "other"},
+                 gcb.MODE_COUNT: {0: "k_count_persistent", 1: "k_count + k_count_hub",
+                                  2: "init phase (round 0)", 3: "rounds"}}[sp.mode_used]
+        if sp.mode_used in (gcb.MODE_EVENT, gcb.MODE_COUNT):
+            cls = 0  # the persistent launch; classes 2-3 (count) / 1-3 (event) are its phases
         name = names[cls]
         kms, kl, kb = sp.kernel_ms[cls], sp.kernel_launches[cls], sp.kernel_bytes[cls]
         achieved = (kb / 1e9) / (kms / 1e3) if kms > 0 else 0.0

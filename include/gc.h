@@ -87,7 +87,7 @@ typedef enum gc_status {
                                       little overhead, so keep it out of timed runs) */
 
 /* Sweep strategy (gc_options.mode).  All modes return identical colours. */
-#define GC_MODE_AUTO 0   /* max-min: SWEEP if max degree <= 32, else EVENT;
+#define GC_MODE_AUTO 0   /* max-min: SWEEP if max degree <= 32, else COUNT;
                             multi-hash and Luby: SWEEP */
 #define GC_MODE_SWEEP 1  /* every round re-scans each uncoloured vertex's row
                             with early exit (the paper's ComputeOp shape) */
@@ -96,6 +96,11 @@ typedef enum gc_status {
                             vertices are re-evaluated; all
                             rounds in one persistent cooperative kernel */
 #define GC_MODE_EVENT_MULTI 3 /* the same method, 4 kernel launches per round */
+#define GC_MODE_COUNT 4  /* work-efficient: per-vertex counts of uncoloured
+                            larger / smaller neighbours; each row is walked
+                            once, when its vertex is coloured (one atomic per
+                            entry); one persistent kernel, one grid barrier
+                            per round */
 
 typedef struct gc_graph gc_graph;
 

@@ -36,7 +36,7 @@ VALIDATE = 1 << 1
 COMPACT = 1 << 2
 OUT_LOCAL_SLICE = 1 << 3
 PROFILE = 1 << 4
-MODE_AUTO, MODE_SWEEP, MODE_EVENT, MODE_EVENT_MULTI = 0, 1, 2, 3
+MODE_AUTO, MODE_SWEEP, MODE_EVENT, MODE_EVENT_MULTI, MODE_COUNT = 0, 1, 2, 3, 4
 
 EXPORTS = ["gc_create_csr", "gc_color", "gc_color_ex", "gc_set_stream", "gc_destroy",
            "gc_last_error", "gc_priorities", "gc_count_colors", "gc_version",

@@ -342,6 +342,13 @@ static void free_scratch(Scratch &s) {
     dfree(s.rstat);
     dfree(s.bitmap);
     dfree(s.hist);
+    dfree(s.cnt);
+    dfree(s.Z);
+    dfree(s.sched);
+    dfree(s.SL);
+    dfree(s.WL);
+    dfree(s.hubs);
+    dfree(s.cctr);
     if (s.host_pinned) hfree(s.host_pinned);
     s = Scratch();
 }
@@ -514,7 +521,7 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
         set_error("gc_color_ex: unknown variant");
         return GC_ERR_INVALID_ARG;
     }
-    if (o->mode < GC_MODE_AUTO || o->mode > GC_MODE_EVENT_MULTI) {
+    if (o->mode < GC_MODE_AUTO || o->mode > GC_MODE_COUNT) {
         set_error("gc_color_ex: unknown mode");
         return GC_ERR_INVALID_ARG;
     }
@@ -527,11 +534,11 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     // and the plain sweep is fastest (measured: 128^3 mesh 0.47 ms sweep vs
     // 0.77 ms event); skewed graphs take thousands of rounds and need the
     // work-efficient event mode (R-MAT s24: 107 ms event vs 1689 ms sweep).
-    if (mode == GC_MODE_AUTO) mode = g->max_deg <= 32 ? GC_MODE_SWEEP : GC_MODE_EVENT;
+    if (mode == GC_MODE_AUTO) mode = g->max_deg <= 32 ? GC_MODE_SWEEP : GC_MODE_COUNT;
     if (luby) mode = GC_MODE_SWEEP;
     if (mode != GC_MODE_SWEEP && H != 1) mode = GC_MODE_SWEEP;
 
-    int rc = ensure_scratch(g, mode != GC_MODE_SWEEP, luby);
+    int rc = ensure_scratch(g, mode == GC_MODE_EVENT || mode == GC_MODE_EVENT_MULTI, luby);
     if (rc) return rc;
     RunParams p;
     p.H = H;
@@ -556,8 +563,20 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
         rc = run_persistent_maxmin(g, p, &res);
     else if (mode == GC_MODE_EVENT_MULTI)
         rc = run_event_maxmin(g, p, &res);
+    else if (mode == GC_MODE_COUNT)
+        rc = g->count_unsafe ? GC_ERR_NOT_SYMMETRIC : run_count_maxmin(g, p, &res);
     else
         rc = run_sweep_maxmin(g, p, &res);
+    if (rc == GC_ERR_NOT_SYMMETRIC && mode == GC_MODE_COUNT) {
+        // The counts need the adjacency MULTISET to be symmetric (a duplicate
+        // entry on one side only, or an asymmetric set, shows up as a count
+        // underflow or a stall -- never as a silently wrong colour, DESIGN.md
+        // 7.0).  The witness kernel only needs the adjacency set: rerun there.
+        g->count_unsafe = true;
+        mode = GC_MODE_EVENT;
+        rc = ensure_scratch(g, true, false);
+        if (!rc) rc = run_persistent_maxmin(g, p, &res);
+    }
     if (rc) {
         cudaEventDestroy(e0);
         cudaEventDestroy(e1);

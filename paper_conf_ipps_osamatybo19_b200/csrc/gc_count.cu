@@ -1,0 +1,777 @@
+// gc_count.cu -- COUNT mode: the max-min colouring (Alg.1 + Alg.5, P:L102-113,
+// P:L506-556; H = 1) computed from per-vertex COUNTS of uncoloured larger and
+// smaller neighbours, all rounds in one persistent cooperative kernel with ONE
+// grid barrier per round.
+//
+// Alg.5 L21-42 make v a local max in round k iff no neighbour u with
+// R[u] > R[v] is still uncoloured at the start of round k (the snapshot of
+// L26, R6), and a local min iff no smaller one is; v takes 2k+1 if min
+// (min wins, R9), else 2k if max.  So with
+//   hi(v) = #{u in adj(v) uncoloured, p(u) > p(v)},  lo(v) = same with <
+// v is coloured in the first round k at whose start hi(v) == 0 or lo(v) == 0.
+// Every vertex coloured in round k decrements, for each neighbour w, hi(w)
+// (if it is larger than w) or lo(w) (if smaller).  A decrement that reaches
+// zero during round k frees that side from round k+1 on: it stamps
+// Z[w].side = k+1 and schedules w for round k+1 (the first stamp wins the
+// schedule bit; a vertex is scheduled exactly once).  Round k+1 then colours
+// its scheduled vertices -- 2(k+1)+1 if Z.lo <= k+1, else 2(k+1) -- and walks
+// their rows.  Decrements of round k+1 stamp k+2, so a concurrent stamp never
+// changes a decision of round k+1: the result is the snapshot result for any
+// interleaving.  Work: the row of every vertex is walked exactly once (when it
+// is coloured) plus one counting pass, so a colouring is O(n + m) with one
+// 8-byte atomic per directed entry; no witness search, no rescans.
+//
+// Kernels: k_count (+ k_count_hub for rows > kHubMin) compute hi/lo of every
+// vertex; k_count_persistent then colours round 0 in a dense init phase and
+// runs rounds k = 0, 1, ... over the scheduled lists:
+//   SL: rows of <= kShortMax entries, one 8-lane group each (4 entries/lane);
+//   WL: longer rows as items of <= kSeg entries, one warp each (8 per lane).
+// Items of round k are the slice [end_{k-1}, end_k) of two monotone arrays
+// (each vertex is scheduled once, so the arrays never wrap).  Appends are
+// staged per block in shared memory (one global atomic per list per block per
+// round).
+
+#include <cstdio>
+#include <cstdlib>
+#include <algorithm>
+
+#include "gc_internal.cuh"
+
+namespace gc {
+
+int ensure_nk(gc_graph *g, int64_t need);
+
+namespace {
+
+constexpr unsigned kFull = 0xFFFFFFFFu;
+constexpr uint32_t kNone = 0xFFFFFFFFu;
+constexpr uint32_t kNever = 0xFFFFFFFFu;  // Z: side never free (yet)
+constexpr int kThreads = 512;              // one block per SM (128 registers)
+constexpr int kShortMax = 32;              // SL rows: one 8-lane group
+constexpr int kSeg = 256;                  // WL item: one warp, 8 entries per lane
+constexpr int kHubMin = 4096;              // k_count: longer rows by blocks
+constexpr int kHubChunk = 4096;
+constexpr uint32_t kFirst = 0x80000000u;   // item flag: colour v in this round
+constexpr unsigned long long kDecHi = 0ull - (1ull << 32);
+constexpr unsigned long long kDecLo = ~0ull;
+
+__device__ __forceinline__ unsigned lane_id() { return threadIdx.x & 31u; }
+
+struct __align__(16) Item {
+    uint32_t v;
+    uint32_t lf;  // entry count | kFirst
+    int64_t e0;   // first entry
+};
+
+// counters (each on its own 128-byte line where it is contended).  The item
+// counts of round k's lists live in slot k % 3: round k reads slot k % 3,
+// appends to slot (k+1) % 3 and clears slot (k+2) % 3 -- the last reader of
+// that slot was round k-1's top, which every block has passed (a reader and
+// a writer of one slot are always separated by a grid barrier).
+enum : int {
+    cS = 0,         // [0, 16, 32]: SL items of the round
+    cW = 48,        // [48, 64, 80]: WL items of the round
+    cK = 96,        // [96, 112, 128]: vertices coloured in the round (stats)
+    cCol = 144,     // vertices coloured so far (host check)
+    cBar = 160,     // barrier arrivals (monotone)
+    cAbort = 176,
+    cErr = 192,     // [192..194] first trap: kind, round, vertex
+    cRounds = 208,  // result: rounds R
+    cIters = 209,   // loop iterations run
+    cVis = 210,     // PROF: entries walked in the rounds
+    cPhaseNs = 211, // PROF: ns in the init phase, the rounds
+    cHubs = 224,    // k_count: hub rows
+    kCCtrWords = 256
+};
+
+struct CArgs {
+    const int64_t *ro;
+    const uint32_t *ci;
+    uint32_t *C;
+    unsigned long long *cnt;  // (hi << 32) | lo
+    uint2 *Z;                 // first round at which the hi / lo side is free
+    uint32_t *sched;          // bit v: v has been scheduled (or coloured in round 0)
+    Item *SL;
+    Item *WL;
+    unsigned long long *ctr;
+    int64_t *nk;
+    int64_t *rstat;
+    int64_t nk_cap;
+    int64_t n;
+    uint32_t key;
+    uint32_t max_rounds;
+    unsigned long long sl_cap, wl_cap;
+};
+
+__device__ __forceinline__ void flag_error(const CArgs &a, unsigned kind, uint32_t k, uint32_t v) {
+    if (atomicCAS(&a.ctr[cErr], 0ull, (unsigned long long)kind) == 0ull) {
+        a.ctr[cErr + 1] = k;
+        a.ctr[cErr + 2] = v;
+    }
+}
+
+__device__ __forceinline__ unsigned long long gtimer() {
+    unsigned long long t;
+    asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+    return t;
+}
+__device__ __forceinline__ unsigned long long ld_acquire(const unsigned long long *p) {
+    unsigned long long v;
+    asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+    return v;
+}
+__device__ __forceinline__ unsigned long long atom_add_release(unsigned long long *p,
+                                                               unsigned long long x) {
+    unsigned long long v;
+    asm volatile("atom.add.release.gpu.global.u64 %0, [%1], %2;" : "=l"(v) : "l"(p), "l"(x) : "memory");
+    return v;
+}
+
+// Grid barrier (cooperative launch: every block is resident): monotone
+// arrival counter, release arrival, acquire spin (which also invalidates the
+// SM's L1, so the next phase sees what other SMs wrote).  A wait beyond 4 s
+// records a trap and makes every block leave instead of hanging the GPU.
+__device__ __forceinline__ bool grid_barrier(const CArgs &a, uint32_t k) {
+    __shared__ int ok_sh;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        int ok = 1;
+        const unsigned long long old = atom_add_release(a.ctr + cBar, 1ull);
+        const unsigned long long target = (old / gridDim.x + 1) * gridDim.x;
+        unsigned spins = 0;
+        const unsigned long long t0 = gtimer();
+        while (ld_acquire(a.ctr + cBar) < target) {
+            if ((++spins & 255u) == 0u) {
+                if (*(volatile unsigned long long *)(a.ctr + cAbort)) {
+                    ok = 0;
+                    break;
+                }
+                if (gtimer() - t0 > 4000000000ull) {
+                    flag_error(a, 100, k, blockIdx.x);
+                    atomicExch(a.ctr + cAbort, 1ull);
+                    ok = 0;
+                    break;
+                }
+            }
+        }
+        ok_sh = ok;
+    }
+    __syncthreads();
+    return ok_sh != 0;
+}
+
+// ---------------------------------------------------------------- staging
+constexpr int kStS = 4096, kStW = 4096, kStF = 4096;
+struct Stage {
+    Item s[kStS];
+    Item w[kStW];
+    uint32_t fresh[kStF];           // vertices this block scheduled in the round
+    unsigned nf;
+    unsigned n[2];
+    unsigned colored;
+    unsigned vis;                   // PROF: entries walked by this block in the round
+    unsigned long long base[2];
+    // append targets of the current round (set by thread 0 at the round top)
+    unsigned long long *cnext[2];   // item-count slots of the next round
+    unsigned long long nbase[2];    // where the next round's items start
+    unsigned long long *ccol;       // coloured-count slot of this round
+};
+constexpr size_t kStageBytes = sizeof(Stage);
+
+__device__ __forceinline__ Stage &stage() {
+    extern __shared__ __align__(16) unsigned char smem_raw[];
+    return *reinterpret_cast<Stage *>(smem_raw);
+}
+
+// Whole warp converged: lanes with `pred` append `val` to staged list li;
+// beyond the shared capacity the entries go straight to the global list.
+__device__ __forceinline__ void stage_append(const CArgs &a, bool pred, const Item &val, int li) {
+    const unsigned m = __ballot_sync(kFull, pred);
+    if (!m) return;
+    Stage &st = stage();
+    const unsigned lane = lane_id();
+    const unsigned leader = __ffs(m) - 1;
+    unsigned base = 0;
+    if (lane == leader) base = atomicAdd(&st.n[li], (unsigned)__popc(m));
+    base = __shfl_sync(kFull, base, leader);
+    const unsigned pos = base + __popc(m & ((1u << lane) - 1u));
+    const unsigned cap = li == 0 ? kStS : kStW;
+    Item *buf = li == 0 ? st.s : st.w;
+    const bool spill = pred && pos >= cap;
+    if (pred && !spill) buf[pos] = val;
+    const unsigned sm = __ballot_sync(kFull, spill);
+    if (sm) {
+        const unsigned sl = __ffs(sm) - 1;
+        unsigned long long gb = 0;
+        if (lane == sl) gb = atomicAdd(st.cnext[li], (unsigned long long)__popc(sm));
+        gb = __shfl_sync(kFull, gb, sl);
+        if (spill) {
+            const unsigned long long at = st.nbase[li] + gb + __popc(sm & ((1u << lane) - 1u));
+            const unsigned long long capg = li == 0 ? a.sl_cap : a.wl_cap;
+            if (at < capg) (li == 0 ? a.SL : a.WL)[at] = val;
+            else flag_error(a, 1, 0, val.v);
+        }
+    }
+}
+
+// Whole block: move staged items to the global lists, add the coloured count.
+// PROF: prs = this round's stat record (entries walked, longest block work).
+__device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullptr,
+                                            unsigned long long t_round = 0) {
+    Stage &st = stage();
+    __syncthreads();
+    if (prs && threadIdx.x == 0) {
+        atomicAdd(reinterpret_cast<unsigned long long *>(prs + 2), (unsigned long long)st.vis);
+        atomicMax(reinterpret_cast<unsigned long long *>(prs + 5), gtimer() - t_round);
+        st.vis = 0;
+    }
+    if (threadIdx.x == 0) {
+        for (int i = 0; i < 2; ++i) {
+            const unsigned c = min(st.n[i], (unsigned)(i == 0 ? kStS : kStW));
+            st.n[i] = c;
+            st.base[i] = c ? st.nbase[i] + atomicAdd(st.cnext[i], (unsigned long long)c) : 0ull;
+            const unsigned long long capg = i == 0 ? a.sl_cap : a.wl_cap;
+            if (c && st.base[i] + c > capg) {
+                flag_error(a, 2, 0, (unsigned)i);
+                st.n[i] = 0;
+            }
+        }
+        st.nf = 0;
+        if (st.colored) {
+            atomicAdd(st.ccol, (unsigned long long)st.colored);
+            atomicAdd(&a.ctr[cCol], (unsigned long long)st.colored);
+        }
+        st.colored = 0;
+    }
+    __syncthreads();
+    for (unsigned i = threadIdx.x; i < st.n[0]; i += blockDim.x) a.SL[st.base[0] + i] = st.s[i];
+    for (unsigned i = threadIdx.x; i < st.n[1]; i += blockDim.x) a.WL[st.base[1] + i] = st.w[i];
+    __syncthreads();
+    if (threadIdx.x < 2) st.n[threadIdx.x] = 0;
+}
+
+// Whole warp converged: schedule the rows of the lanes with `pred` (vertex w,
+// row [rs, rs + len)) for the next round: short rows as one SL item, longer
+// rows as ceil(len / kSeg) WL items (expanded by the whole warp).
+__device__ __noinline__ void schedule_rows(const CArgs &a, bool pred, uint32_t w, int64_t rs,
+                                              int64_t len, bool first) {
+    const uint32_t ff = first ? kFirst : 0u;
+    const bool shortrow = pred && len <= kShortMax;
+    Item it;
+    it.v = w;
+    it.lf = (uint32_t)len | ff;
+    it.e0 = rs;
+    stage_append(a, shortrow, it, 0);
+    unsigned lm = __ballot_sync(kFull, pred && !shortrow);
+    while (lm) {
+        const int src = __ffs(lm) - 1;
+        lm &= lm - 1;
+        const uint32_t ww = __shfl_sync(kFull, w, src);
+        const int64_t r0 = __shfl_sync(kFull, rs, src);
+        const int64_t ln = __shfl_sync(kFull, len, src);
+        const uint32_t nseg = (uint32_t)((ln + kSeg - 1) / kSeg);
+        for (uint32_t q0 = 0; q0 < nseg; q0 += 32) {
+            const uint32_t q = q0 + lane_id();
+            Item si;
+            si.v = ww;
+            const int64_t e0 = r0 + (int64_t)q * kSeg;
+            si.e0 = e0;
+            si.lf = (uint32_t)min((int64_t)kSeg, r0 + ln - e0) | (q == 0 ? ff : 0u);
+            stage_append(a, q < nseg, si, 1);
+        }
+    }
+}
+
+// Colour v in round k (its scheduled round): min (2k+1) if the lo side is
+// free at the start of round k, else max (2k) -- Alg.5 L37-42, R9.
+__device__ __forceinline__ void colour(const CArgs &a, uint32_t v, uint32_t k) {
+    const uint2 z = a.Z[v];
+    const bool lo_free = z.y <= k, hi_free = z.x <= k;
+    if (!lo_free && !hi_free) flag_error(a, 3, k, v);
+    a.C[v] = 2u * k + (lo_free ? 1u : 0u);
+}
+
+// Walk entries e, e + stride, ... (< end, Q of them) of the row of v coloured
+// in round k (v == kNone: idle lane; whole warp converged): decrement the
+// side of each neighbour w that v belongs to; a side reaching zero is free
+// from round k+1 and schedules w (first time only).
+template <int Q>
+__device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, int64_t e,
+                                     int64_t end, int stride, uint32_t k, uint32_t &nvis) {
+    uint32_t w[Q];
+#pragma unroll
+    for (int q = 0; q < Q; ++q) {
+        const int64_t eq = e + (int64_t)q * stride;
+        w[q] = (v != kNone && eq < end) ? __ldcs(a.ci + eq) : kNone;
+    }
+    unsigned long long old[Q];
+    bool hi[Q];
+#pragma unroll
+    for (int q = 0; q < Q; ++q) {
+        hi[q] = false;
+        old[q] = 0;
+        if (w[q] != kNone) {
+            hi[q] = pv > weight_mix(w[q] ^ a.key);  // v is a larger neighbour of w
+            old[q] = atomicAdd(&a.cnt[w[q]], hi[q] ? kDecHi : kDecLo);
+        }
+    }
+    bool fresh[Q];
+#pragma unroll
+    for (int q = 0; q < Q; ++q) {
+        fresh[q] = false;
+        if (w[q] != kNone) {
+            ++nvis;
+            const uint32_t side = hi[q] ? (uint32_t)(old[q] >> 32) : (uint32_t)old[q];
+            if (side == 1u) {
+                reinterpret_cast<uint32_t *>(a.Z + w[q])[hi[q] ? 0 : 1] = k + 1u;
+                const uint32_t bit = 1u << (w[q] & 31u);
+                fresh[q] = (atomicOr(&a.sched[w[q] >> 5], bit) & bit) == 0u;
+            } else if (side == 0u) {
+                flag_error(a, 4, k, w[q]);  // count underflow: adjacency not symmetric
+            }
+        }
+    }
+    // (rare) newly scheduled neighbours go to the block's fresh list; their
+    // rows are fetched once per block at the end of the round (schedule_fresh)
+    // instead of one dependent load per q here
+    bool ovf[Q];
+#pragma unroll
+    for (int q = 0; q < Q; ++q) {
+        ovf[q] = false;
+        if (fresh[q]) {
+            const unsigned pos = atomicAdd(&stage().nf, 1u);
+            if (pos < (unsigned)kStF) stage().fresh[pos] = w[q];
+            else ovf[q] = true;
+        }
+    }
+#pragma unroll
+    for (int q = 0; q < Q; ++q) {
+        if (__any_sync(kFull, ovf[q])) {  // shared list full: schedule here
+            int64_t rs = 0, re = 0;
+            if (ovf[q]) {
+                rs = a.ro[w[q]];
+                re = a.ro[w[q] + 1];
+            }
+            schedule_rows(a, ovf[q], w[q], rs, re - rs, true);
+        }
+    }
+}
+
+// Whole block, end of a round: stage the items of the vertices on the fresh
+// list (all their row offsets are fetched in one dependent step).
+__device__ __forceinline__ void schedule_fresh(const CArgs &a) {
+    Stage &st = stage();
+    __syncthreads();
+    const unsigned nf = min(st.nf, (unsigned)kStF);
+    const unsigned wib = threadIdx.x >> 5, nwb = blockDim.x >> 5;
+    for (unsigned base = wib * 32; base < nf; base += nwb * 32) {
+        const unsigned idx = base + lane_id();
+        const bool valid = idx < nf;
+        uint32_t w = 0;
+        int64_t rs = 0, re = 0;
+        if (valid) {
+            w = st.fresh[idx];
+            rs = a.ro[w];
+            re = a.ro[w + 1];
+        }
+        schedule_rows(a, valid, w, rs, re - rs, true);
+    }
+}
+
+// Thread 0 of each block: append targets of round k (see the counter enum).
+__device__ __forceinline__ void set_targets(const CArgs &a, uint32_t k, unsigned long long sbase_next,
+                                            unsigned long long wbase_next) {
+    Stage &st = stage();
+    if (threadIdx.x == 0) {
+        const int nx = (int)((k + 1) % 3);
+        st.cnext[0] = a.ctr + cS + 16 * nx;
+        st.cnext[1] = a.ctr + cW + 16 * nx;
+        st.nbase[0] = sbase_next;
+        st.nbase[1] = wbase_next;
+        st.ccol = a.ctr + cK + 16 * (int)(k % 3);
+    }
+    __syncthreads();
+}
+
+template <bool PROF>
+__global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
+    const unsigned lane = lane_id();
+    const unsigned long long gtid = (unsigned long long)blockIdx.x * blockDim.x + threadIdx.x;
+    const unsigned long long nthreads = (unsigned long long)gridDim.x * blockDim.x;
+    const unsigned long long gwarp = gtid >> 5, nwarps = nthreads >> 5;
+    const int64_t n = a.n;
+    uint32_t nvis = 0;
+    unsigned long long nvis_tot = 0, t_rounds = 0;
+    unsigned long long t0 = PROF ? gtimer() : 0ull;
+    {
+        Stage &st = stage();
+        if (threadIdx.x < 2) st.n[threadIdx.x] = 0;
+        if (threadIdx.x == 0) st.colored = 0;
+        if (threadIdx.x == 0) st.vis = 0;
+        if (threadIdx.x == 0) st.nf = 0;
+        // init appends round 0's items to slot 0 at position 0; its colourings
+        // count for round 0 (so the "next round" targets are round 0's here)
+        if (threadIdx.x == 0) {
+            st.cnext[0] = a.ctr + cS;
+            st.cnext[1] = a.ctr + cW;
+            st.nbase[0] = st.nbase[1] = 0ull;
+            st.ccol = a.ctr + cK;
+        }
+        __syncthreads();
+    }
+    // ---------------------------------------------------- init = round 0
+    // lane per vertex, 32 consecutive vertices per warp (one sched word)
+    for (unsigned long long base = gwarp * 32; base < (unsigned long long)n; base += nwarps * 32) {
+        const uint32_t v = (uint32_t)(base + lane);
+        const bool valid = (int64_t)(base + lane) < n;
+        const unsigned long long c = valid ? a.cnt[v] : 0x100000001ull;
+        const uint32_t hi = (uint32_t)(c >> 32), lo = (uint32_t)c;
+        const bool zero = valid && (hi == 0u || lo == 0u);
+        int64_t rs = 0, re = 0;
+        if (valid) {
+            a.Z[v] = make_uint2(hi == 0u ? 0u : kNever, lo == 0u ? 0u : kNever);
+            a.C[v] = zero ? (lo == 0u ? 1u : 0u) : GC_UNC;  // round 0: min wins (R9)
+            if (zero) {
+                rs = a.ro[v];
+                re = a.ro[v + 1];
+            }
+        }
+        const unsigned word = __ballot_sync(kFull, zero);
+        if (lane == 0) {
+            a.sched[base >> 5] = word;
+            if (word) atomicAdd(&stage().colored, (unsigned)__popc(word));
+        }
+        schedule_rows(a, zero && re > rs, v, rs, re - rs, false);  // walked in round 0
+    }
+    stage_flush(a);
+    if (!grid_barrier(a, 0)) return;
+    if (PROF && gtid == 0) {
+        const unsigned long long t = gtimer();
+        a.ctr[cPhaseNs] = t - t0;
+        t0 = t;
+    }
+    // ------------------------------------------------------------ rounds
+    unsigned long long sl0 = 0, wl0 = 0;  // where round k's items start
+    int64_t rem = n;                      // gtid 0 only: uncoloured at the round start
+    uint32_t last = 0;                    // last round with a colouring
+    uint32_t k = 0;
+    for (;; ++k) {
+        const int cur = (int)(k % 3);
+        const unsigned long long ns = __ldcg(&a.ctr[cS + 16 * cur]), nw = __ldcg(&a.ctr[cW + 16 * cur]);
+        if (gtid == 0) {
+            if (k > 0) {
+                const int prv = (int)((k + 2) % 3);
+                rem -= (int64_t)__ldcg(&a.ctr[cK + 16 * prv]);
+                a.ctr[cK + 16 * prv] = 0ull;  // only gtid 0 reads these slots
+            }
+            if ((int64_t)k < a.nk_cap) a.nk[k] = rem;
+            if (PROF && k > 0 && (int64_t)(k - 1) < a.nk_cap) a.rstat[16 * (k - 1) + 3] = a.nk[k - 1] - rem;
+            const int nxt2 = (int)((k + 2) % 3);
+            a.ctr[cS + 16 * nxt2] = 0ull;  // slot of round k+2 (last read at round k-1's top)
+            a.ctr[cW + 16 * nxt2] = 0ull;
+        }
+        if (__ldcg(&a.ctr[cErr]) != 0ull) break;  // a trap fired (uniform: read after a barrier)
+        if (ns == 0 && nw == 0) break;            // nothing scheduled: done
+        if (k >= a.max_rounds) break;
+        if (k > 0) last = k;  // every item of round k >= 1 colours (kFirst)
+        if (PROF && gtid == 0 && (int64_t)k < a.nk_cap) {
+            a.rstat[16 * k + 0] = (int64_t)ns;
+            a.rstat[16 * k + 1] = (int64_t)nw;
+        }
+        const unsigned long long sl1 = sl0 + ns, wl1 = wl0 + nw;
+        const unsigned long long t_round = PROF ? gtimer() : 0ull;
+        set_targets(a, k, sl1, wl1);
+        // short rows: 4 per warp, 8 lanes each, 4 entries per lane
+        for (unsigned long long b = sl0 + gwarp * 4; b < sl1; b += nwarps * 4) {
+            const unsigned long long idx = b + (lane >> 3);
+            uint32_t v = kNone, len = 0, pv = 0;
+            int64_t e0 = 0;
+            if (idx < sl1) {
+                const Item it = a.SL[idx];
+                v = it.v;
+                len = it.lf & ~kFirst;
+                e0 = it.e0;
+                pv = weight_mix(v ^ a.key);
+                if ((it.lf & kFirst) && (lane & 7u) == 0u) {
+                    colour(a, v, k);
+                    atomicAdd(&stage().colored, 1u);
+                }
+            }
+            walk<4>(a, v, pv, e0 + (lane & 7u), e0 + len, 8, k, nvis);
+        }
+        // longer rows: one <= kSeg-entry item per warp
+        for (unsigned long long i = wl0 + gwarp; i < wl1; i += nwarps) {
+            const Item it = a.WL[i];
+            const uint32_t pv = weight_mix(it.v ^ a.key);
+            if ((it.lf & kFirst) && lane == 0) {
+                colour(a, it.v, k);
+                atomicAdd(&stage().colored, 1u);
+            }
+            walk<kSeg / 32>(a, it.v, pv, it.e0 + lane, it.e0 + (it.lf & ~kFirst), 32, k, nvis);
+        }
+        sl0 = sl1;
+        wl0 = wl1;
+        if (PROF) {
+            const unsigned s = __reduce_add_sync(kFull, nvis);
+            if (lane == 0 && s) atomicAdd(&stage().vis, s);
+            nvis_tot += nvis;
+            nvis = 0;
+        }
+        schedule_fresh(a);
+        stage_flush(a, (PROF && (int64_t)k < a.nk_cap) ? a.rstat + 16 * k : nullptr, t_round);
+        if (!grid_barrier(a, k)) return;
+        if (PROF && gtid == 0) {
+            const unsigned long long t = gtimer();
+            if ((int64_t)k < a.nk_cap) a.rstat[16 * k + 4] = (int64_t)(t - t0);
+            t_rounds += t - t0;
+            t0 = t;
+        }
+    }
+    if (gtid == 0) {
+        a.ctr[cRounds] = n > 0 ? last + 1 : 0;
+        a.ctr[cIters] = k;
+        if (PROF) a.ctr[cPhaseNs + 1] = t_rounds;
+    }
+    if (PROF) {
+        const unsigned long long s = __reduce_add_sync(kFull, (unsigned)nvis_tot);
+        if (lane == 0 && s) atomicAdd(&a.ctr[cVis], s);
+    }
+}
+
+// hi / lo counts of every vertex (round-0 state: everything is uncoloured).
+// A warp takes 32 consecutive vertices: rows <= 16 one lane each, rows up to
+// kHubMin the whole warp (coalesced), longer rows go to the hub list.
+__global__ void __launch_bounds__(256) k_count(const int64_t *__restrict__ ro,
+                                               const uint32_t *__restrict__ ci, int64_t n,
+                                               uint32_t key, unsigned long long *cnt,
+                                               uint2 *hubs, unsigned long long *nhubs) {
+    const unsigned lane = lane_id();
+    const unsigned long long gw = ((unsigned long long)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+    const unsigned long long nw = ((unsigned long long)gridDim.x * blockDim.x) >> 5;
+    for (unsigned long long base = gw * 32; base < (unsigned long long)n; base += nw * 32) {
+        const int64_t v = (int64_t)(base + lane);
+        const bool valid = v < n;
+        int64_t rs = 0, re = 0;
+        if (valid) {
+            rs = ro[v];
+            re = ro[v + 1];
+        }
+        const int64_t deg = re - rs;
+        const uint32_t pv = weight_mix((uint32_t)v ^ key);
+        if (valid && deg <= 16) {
+            uint32_t h = 0;
+            uint32_t u[16];
+#pragma unroll
+            for (int q = 0; q < 16; ++q) u[q] = q < deg ? __ldcs(ci + rs + q) : 0u;
+#pragma unroll
+            for (int q = 0; q < 16; ++q) h += (q < deg && weight_mix(u[q] ^ key) > pv) ? 1u : 0u;
+            cnt[v] = ((unsigned long long)h << 32) | (unsigned long long)(deg - h);
+        }
+        const bool big = valid && deg > kHubMin;
+        if (big) {
+            cnt[v] = 0ull;  // k_count_hub adds the chunks
+            const int64_t nch = (deg + kHubChunk - 1) / kHubChunk;
+            const unsigned long long b = atomicAdd(nhubs, (unsigned long long)nch);
+            for (int64_t c = 0; c < nch; ++c)
+                hubs[b + c] = make_uint2((uint32_t)v, (uint32_t)c);
+        }
+        unsigned mid = __ballot_sync(kFull, valid && deg > 16 && deg <= kHubMin);
+        while (mid) {
+            const int src = __ffs(mid) - 1;
+            mid &= mid - 1;
+            const int64_t r0 = __shfl_sync(kFull, rs, src), r1 = __shfl_sync(kFull, re, src);
+            const uint32_t p = __shfl_sync(kFull, pv, src);
+            uint32_t h = 0;
+            for (int64_t e = r0 + lane; e < r1; e += 128) {
+                uint32_t u[4];
+#pragma unroll
+                for (int q = 0; q < 4; ++q) u[q] = e + 32 * q < r1 ? __ldcs(ci + e + 32 * q) : 0u;
+#pragma unroll
+                for (int q = 0; q < 4; ++q)
+                    h += (e + 32 * q < r1 && weight_mix(u[q] ^ key) > p) ? 1u : 0u;
+            }
+            h = __reduce_add_sync(kFull, h);
+            if (lane == (unsigned)src)
+                cnt[v] = ((unsigned long long)h << 32) | (unsigned long long)(deg - h);
+        }
+    }
+}
+
+// Rows longer than kHubMin: one block per kHubChunk-entry chunk (the chunk
+// list (v, c) was written by k_count); partial counts are added atomically.
+__global__ void __launch_bounds__(256) k_count_hub(const int64_t *__restrict__ ro,
+                                                   const uint32_t *__restrict__ ci, uint32_t key,
+                                                   unsigned long long *cnt, const uint2 *hubs,
+                                                   const unsigned long long *nhubs) {
+    __shared__ uint32_t red[8];
+    const unsigned long long nh = *nhubs;
+    for (unsigned long long i = blockIdx.x; i < nh; i += gridDim.x) {
+        const uint2 hc = hubs[i];
+        const uint32_t v = hc.x;
+        const int64_t rs = ro[v], re = ro[v + 1];
+        const uint32_t pv = weight_mix(v ^ key);
+        const int64_t c0 = rs + (int64_t)hc.y * kHubChunk, c1 = min(re, c0 + (int64_t)kHubChunk);
+        uint32_t hcount = 0;
+#pragma unroll 4
+        for (int64_t e = c0 + threadIdx.x; e < c1; e += blockDim.x)
+            hcount += weight_mix(__ldcs(ci + e) ^ key) > pv ? 1u : 0u;
+        hcount = __reduce_add_sync(kFull, hcount);
+        if (lane_id() == 0) red[threadIdx.x >> 5] = hcount;
+        __syncthreads();
+        if (threadIdx.x == 0) {
+            uint32_t t = 0;
+            for (int j = 0; j < (int)(blockDim.x >> 5); ++j) t += red[j];
+            const unsigned long long tot = (unsigned long long)(c1 - c0);
+            atomicAdd(&cnt[v], ((unsigned long long)t << 32) + (tot - t));
+        }
+        __syncthreads();
+    }
+}
+
+template <bool PROF>
+int launch(gc_graph *g, CArgs &a, int *blocks_out) {
+    int per_sm = 0;
+    GC_CUDA_TRY(cudaFuncSetAttribute(k_count_persistent<PROF>,
+                                     cudaFuncAttributeMaxDynamicSharedMemorySize, (int)kStageBytes));
+    GC_CUDA_TRY(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_count_persistent<PROF>,
+                                                              kThreads, kStageBytes));
+    if (per_sm < 1) {
+        set_error("persistent count kernel cannot be resident");
+        return GC_ERR_CUDA;
+    }
+    const int blocks = per_sm * g->sm_count;
+    void *args[] = {&a};
+    GC_CUDA_TRY(cudaLaunchCooperativeKernel((void *)k_count_persistent<PROF>, blocks, kThreads, args,
+                                            kStageBytes, g->stream));
+    *blocks_out = blocks;
+    return GC_OK;
+}
+
+}  // namespace
+
+// Scratch of COUNT mode (allocated on first use, kept with the handle).
+int ensure_count_scratch(gc_graph *g) {
+    Scratch &s = g->s;
+    const size_t nn = (size_t)std::max<int64_t>(g->n, 1);
+    if (s.cnt) return GC_OK;
+    GC_CUDA_TRY(dmalloc(&s.cnt, nn * 8));
+    GC_CUDA_TRY(dmalloc(&s.Z, nn * 8));
+    GC_CUDA_TRY(dmalloc(&s.sched, ((nn + 31) / 32) * 4));
+    s.sl_cap = (int64_t)nn;
+    s.wl_cap = (int64_t)nn + g->nnz / kSeg + 1;
+    GC_CUDA_TRY(dmalloc(&s.SL, (size_t)s.sl_cap * sizeof(Item)));
+    GC_CUDA_TRY(dmalloc(&s.WL, (size_t)s.wl_cap * sizeof(Item)));
+    // hub chunk list: at most nnz / kHubChunk entries
+    GC_CUDA_TRY(dmalloc(&s.hubs, ((size_t)g->nnz / kHubChunk + 1) * 8));
+    GC_CUDA_TRY(dmalloc(&s.cctr, kCCtrWords * sizeof(unsigned long long)));
+    return GC_OK;
+}
+
+int run_count_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
+    Scratch &s = g->s;
+    const int64_t n = g->n;
+    r->rounds = r->inner = r->launches = 0;
+    if (n == 0) return GC_OK;
+    int rc = ensure_count_scratch(g);
+    if (rc) return rc;
+    const int64_t max_rounds = std::min<int64_t>(std::min<int64_t>(p.max_rounds, 0xFFFFFFF0ll),
+                                                 n / 2 + 2);
+    rc = ensure_nk(g, std::min<int64_t>(std::min<int64_t>(n + 2, max_rounds + 2), 1 << 20));
+    if (rc) return rc;
+    cudaStream_t st = g->stream;
+    GC_CUDA_TRY(cudaMemsetAsync(s.cctr, 0, kCCtrWords * sizeof(unsigned long long), st));
+    const bool prof = p.prof && p.prof->on;
+    cudaEvent_t e0 = nullptr, e1 = nullptr, e2 = nullptr;
+    if (prof) {
+        GC_CUDA_TRY(cudaEventCreate(&e0));
+        GC_CUDA_TRY(cudaEventCreate(&e1));
+        GC_CUDA_TRY(cudaEventCreate(&e2));
+        GC_CUDA_TRY(cudaEventRecord(e0, st));
+    }
+    const uint32_t key = p.keys.k[0];
+    unsigned long long *nhubs = s.cctr + cHubs;
+    {
+        const int64_t warps = (n + 31) / 32;
+        const int blocks = (int)std::min<int64_t>((warps + 7) / 8, (int64_t)g->sm_count * 16);
+        uint2 *hubs = reinterpret_cast<uint2 *>(s.hubs);
+        k_count<<<blocks, 256, 0, st>>>(g->ro, g->ci, n, key, s.cnt, hubs, nhubs);
+        k_count_hub<<<g->sm_count * 8, 256, 0, st>>>(g->ro, g->ci, key, s.cnt, hubs, nhubs);
+        GC_CUDA_TRY(cudaGetLastError());
+    }
+    if (prof) GC_CUDA_TRY(cudaEventRecord(e1, st));
+    CArgs a;
+    a.ro = g->ro;
+    a.ci = g->ci;
+    a.C = s.C;
+    a.cnt = s.cnt;
+    a.Z = reinterpret_cast<uint2 *>(s.Z);
+    a.sched = s.sched;
+    a.SL = reinterpret_cast<Item *>(s.SL);
+    a.WL = reinterpret_cast<Item *>(s.WL);
+    a.ctr = s.cctr;
+    a.nk = s.nk;
+    a.rstat = s.rstat;
+    a.nk_cap = s.nk_cap;
+    a.n = n;
+    a.key = key;
+    a.max_rounds = (uint32_t)max_rounds;
+    a.sl_cap = (unsigned long long)s.sl_cap;
+    a.wl_cap = (unsigned long long)s.wl_cap;
+    if (prof) GC_CUDA_TRY(cudaMemsetAsync(s.rstat, 0, sizeof(int64_t) * 16 * (size_t)s.nk_cap, st));
+    int blocks = 0;
+    rc = prof ? launch<true>(g, a, &blocks) : launch<false>(g, a, &blocks);
+    if (rc) return rc;
+    r->launches += 3;  // k_count, k_count_hub, persistent kernel
+    if (prof) GC_CUDA_TRY(cudaEventRecord(e2, st));
+    unsigned long long h[kCCtrWords];
+    GC_CUDA_TRY(cudaMemcpyAsync(h, s.cctr, sizeof(h), cudaMemcpyDeviceToHost, st));
+    GC_CUDA_TRY(cudaStreamSynchronize(st));
+    if (h[cErr] != 0) {
+        char buf[200];
+        if (h[cErr] == 4)
+            snprintf(buf, sizeof(buf), "count underflow at vertex %llu in round %llu: the adjacency is "
+                     "not symmetric", h[cErr + 2], h[cErr + 1]);
+        else
+            snprintf(buf, sizeof(buf), "internal consistency check %llu failed in round %llu (vertex %llu)",
+                     h[cErr], h[cErr + 1], h[cErr + 2]);
+        set_error(buf);
+        return h[cErr] == 4 ? GC_ERR_NOT_SYMMETRIC : GC_ERR_CUDA;
+    }
+    if (h[cCol] != (unsigned long long)n) {
+        set_error("max-min colouring stalled with uncoloured vertices: the adjacency is not symmetric");
+        return GC_ERR_NOT_SYMMETRIC;
+    }
+    r->rounds = (int64_t)h[cRounds];
+    r->inner = r->rounds;
+    if (prof) {
+        float ms_all = 0.f, ms_cnt = 0.f;
+        cudaEventElapsedTime(&ms_all, e0, e2);
+        cudaEventElapsedTime(&ms_cnt, e0, e1);
+        cudaEventDestroy(e0);
+        cudaEventDestroy(e1);
+        cudaEventDestroy(e2);
+        // class 0: the persistent kernel; 1: counting kernels; 2: its init
+        // phase (round 0); 3: its rounds (globaltimer, block 0)
+        p.prof->ms[0] += ms_all - ms_cnt;
+        p.prof->launches[0] += 1;
+        p.prof->launch_us.push_back(1e3f * (ms_all - ms_cnt));
+        p.prof->ms[1] += ms_cnt;
+        p.prof->launches[1] += 2;
+        p.prof->ms[2] += (double)h[cPhaseNs] / 1e6;
+        p.prof->ms[3] += (double)h[cPhaseNs + 1] / 1e6;
+        // algorithmic bytes.  Counting: 8 B offsets + 8 B
+        // count per vertex + 4 B per entry.  Persistent kernel: init 8 B
+        // count + 8 B Z + 4 B colour + 8 B offsets (coloured in round 0) per
+        // vertex + n/8 B schedule bits; per scheduled vertex 16 B item write
+        // + 16 B item read + 8 B offsets + 8 B Z + 4 B colour; per walked
+        // entry 4 B column id + 8 B count read + 8 B count write.
+        const int64_t vis = (int64_t)h[cVis];
+        const int64_t m = g->nnz;
+        p.prof->bytes[1] += 16 * n + 4 * m;
+        p.prof->bytes[0] += 28 * n + n / 8 + 52 * n + 20 * vis;
+        p.prof->visits += vis;
+    }
+    return GC_OK;
+}
+
+}  // namespace gc

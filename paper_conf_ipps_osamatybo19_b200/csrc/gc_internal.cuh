@@ -61,6 +61,15 @@ struct Scratch {
     unsigned long long *hist = nullptr;  // GC_PROFILE_HIST histograms (gc_persist.cu)
     int64_t bitmap_words = 0;
     int64_t *host_pinned = nullptr;  // pinned readback area
+    // COUNT mode (gc_count.cu)
+    unsigned long long *cnt = nullptr;   // (hi << 32) | lo uncoloured-neighbour counts
+    uint32_t *Z = nullptr;               // uint2 per vertex: round from which hi / lo is free
+    uint32_t *sched = nullptr;           // scheduled bit per vertex
+    void *SL = nullptr;                  // short-row items (16 B)
+    void *WL = nullptr;                  // long-row segment items (16 B)
+    uint32_t *hubs = nullptr;            // k_count: rows counted by blocks
+    unsigned long long *cctr = nullptr;  // counters of the persistent count kernel
+    int64_t sl_cap = 0, wl_cap = 0;
 };
 
 }  // namespace gc
@@ -79,6 +88,7 @@ struct gc_graph {
     gc::Scratch s;
     gc::Dist *dist = nullptr;
     int sm_count = 148;
+    bool count_unsafe = false;  // COUNT mode saw an asymmetric multiset: use EVENT
 };
 
 namespace gc {
@@ -177,6 +187,7 @@ int ensure_scratch(gc_graph *g, bool need_event, bool need_luby);
 int run_sweep_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int run_event_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
+int run_count_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int run_luby(gc_graph *g, const RunParams &p, RunResult *r);
 int64_t count_colors_device(gc_graph *g, const uint32_t *C, int64_t n, bool compact,
                             uint32_t *C_inout, int64_t *launches);

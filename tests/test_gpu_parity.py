@@ -21,7 +21,7 @@ from paper_conf_ipps_osamatybo19_b200 import build as gbuild
 
 pytestmark = pytest.mark.gpu
 
-MODES = [gcb.MODE_SWEEP, gcb.MODE_EVENT, gcb.MODE_EVENT_MULTI]
+MODES = [gcb.MODE_SWEEP, gcb.MODE_EVENT, gcb.MODE_EVENT_MULTI, gcb.MODE_COUNT]
 
 
 @pytest.fixture(scope="module", autouse=True)

@@ -12,7 +12,8 @@ ap.add_argument("--scale", type=int, default=24)
 ap.add_argument("--variant", default="maxmin")
 ap.add_argument("--warm", action="store_true")
 a = ap.parse_args()
-mode = {"event": gcb.MODE_EVENT, "sweep": gcb.MODE_SWEEP, "multi": gcb.MODE_EVENT_MULTI}[a.mode]
+mode = {"event": gcb.MODE_EVENT, "sweep": gcb.MODE_SWEEP, "multi": gcb.MODE_EVENT_MULTI,
+        "count": gcb.MODE_COUNT}[a.mode]
 var = {"maxmin": gcb.MAXMIN, "luby": gcb.LUBY_MIS, "multihash": gcb.MULTIHASH(4)}[a.variant]
 g = G.rmat(a.scale, 16, seed=1, device="cuda")
 torch.cuda.synchronize()

@@ -23,7 +23,8 @@ def main():
     ap.add_argument("--out", default="gpurun_out/rounds.json")
     a = ap.parse_args()
     g = G.rmat(a.scale, 16, seed=1, device="cuda")
-    mode = {"event": gcb.MODE_EVENT, "sweep": gcb.MODE_SWEEP, "multi": gcb.MODE_EVENT_MULTI}[a.mode]
+    mode = {"event": gcb.MODE_EVENT, "sweep": gcb.MODE_SWEEP, "multi": gcb.MODE_EVENT_MULTI,
+            "count": gcb.MODE_COUNT}[a.mode]
     out = torch.empty(g.n, dtype=torch.int32, device="cuda")
     hist_path = a.out + ".hist"
     if os.path.exists(hist_path):
@@ -34,13 +35,18 @@ def main():
         _, k, st = h.color(1, gcb.MAXMIN, out, mode=mode, flags=gcb.PROFILE, stats=True,
                            trace_cap=1 << 15)
     R = st.rounds
-    per = {gcb.MODE_EVENT: 3, gcb.MODE_EVENT_MULTI: 4}.get(mode, 2)
+    per = {gcb.MODE_EVENT: 3, gcb.MODE_EVENT_MULTI: 4, gcb.MODE_COUNT: 1}.get(mode, 2)
     lu = st.launch_us
     rows = []
     for r in range(R):
         rs = st.round_stats[16 * r: 16 * r + 16]
         # persistent kernel: per-phase times (ns) are in the round record
-        t = [x / 1e3 for x in rs[4:7]] if mode == gcb.MODE_EVENT else lu[per * r: per * r + per]
+        if mode == gcb.MODE_COUNT:  # [SL items, WL items, entries, coloured, round ns, max block ns]
+            t = [rs[4] / 1e3]
+        elif mode == gcb.MODE_EVENT:
+            t = [x / 1e3 for x in rs[4:7]]
+        else:
+            t = lu[per * r: per * r + per]
         rows.append({"k": r, "us": t, "stats": rs})
     buckets = [(0, 1), (1, 2), (2, 10), (10, 100), (100, 500), (500, 1000), (1000, 2000),
                (2000, R)]
