@@ -344,7 +344,6 @@ static void free_scratch(Scratch &s) {
     dfree(s.hist);
     dfree(s.cnt);
     dfree(s.Z);
-    dfree(s.sched);
     dfree(s.SL);
     dfree(s.WL);
     dfree(s.hubs);

@@ -10,22 +10,26 @@
 //   hi(v) = #{u in adj(v) uncoloured, p(u) > p(v)},  lo(v) = same with <
 // v is coloured in the first round k at whose start hi(v) == 0 or lo(v) == 0.
 // Every vertex coloured in round k decrements, for each neighbour w, hi(w)
-// (if it is larger than w) or lo(w) (if smaller).  A decrement that reaches
-// zero during round k frees that side from round k+1 on: it stamps
-// Z[w].side = k+1 and schedules w for round k+1 (the first stamp wins the
-// schedule bit; a vertex is scheduled exactly once).  Round k+1 then colours
-// its scheduled vertices -- 2(k+1)+1 if Z.lo <= k+1, else 2(k+1) -- and walks
-// their rows.  Decrements of round k+1 stamp k+2, so a concurrent stamp never
-// changes a decision of round k+1: the result is the snapshot result for any
-// interleaving.  Work: the row of every vertex is walked exactly once (when it
-// is coloured) plus one counting pass, so a colouring is O(n + m) with one
-// 8-byte atomic per directed entry; no witness search, no rescans.
+// (if it is larger than w) or lo(w) (if smaller), both halves of ONE 64-bit
+// word, so the atomic returns both counts: the decrement that takes a side to
+// zero while the other side is still positive is the unique first freeing of
+// w -- it schedules w for round k+1 (w is min-coloured there if the freed side
+// is lo).  If the other side is already zero, w was scheduled earlier; a lo
+// side freed second stamps Zlo[w] = k+1, so a w scheduled by its hi side in
+// round k still takes the min colour when lo was freed in the same round
+// (min wins, Alg.5 L37-42, R9), and a stamp of round k+1 (k+2) never changes a
+// decision of round k+1: the result is the snapshot result (Alg.5 L26, R6)
+// for any interleaving.  Work: the row of every vertex is walked exactly once
+// (when it is coloured) plus one counting pass, so a colouring is O(n + m)
+// with one 8-byte atomic per directed entry; no witness search, no rescans.
 //
 // Kernels: k_count (+ k_count_hub for rows > kHubMin) compute hi/lo of every
 // vertex; k_count_persistent then colours round 0 in a dense init phase and
 // runs rounds k = 0, 1, ... over the scheduled lists:
 //   SL: rows of <= kShortMax entries, one 8-lane group each (4 entries/lane);
 //   WL: longer rows as items of <= kSeg entries, one warp each (8 per lane).
+// Work units (WL items, groups of 4 SL items) are dealt round-robin over the
+// blocks, so every SM gets an equal share of a round's few thousand units.
 // Items of round k are the slice [end_{k-1}, end_k) of two monotone arrays
 // (each vertex is scheduled once, so the arrays never wrap).  Appends are
 // staged per block in shared memory (one global atomic per list per block per
@@ -52,6 +56,8 @@ constexpr int kSeg = 256;                  // WL item: one warp, 8 entries per l
 constexpr int kHubMin = 4096;              // k_count: longer rows by blocks
 constexpr int kHubChunk = 4096;
 constexpr uint32_t kFirst = 0x80000000u;   // item flag: colour v in this round
+constexpr uint32_t kLoSide = 0x40000000u;  // item flag: scheduled by its lo side (min colour)
+constexpr uint32_t kLenMask = 0x3FFFFFFFu;
 constexpr unsigned long long kDecHi = 0ull - (1ull << 32);
 constexpr unsigned long long kDecLo = ~0ull;
 
@@ -59,7 +65,7 @@ __device__ __forceinline__ unsigned lane_id() { return threadIdx.x & 31u; }
 
 struct __align__(16) Item {
     uint32_t v;
-    uint32_t lf;  // entry count | kFirst
+    uint32_t lf;  // entry count | kFirst | kLoSide
     int64_t e0;   // first entry
 };
 
@@ -72,7 +78,7 @@ enum : int {
     cS = 0,         // [0, 16, 32]: SL items of the round
     cW = 48,        // [48, 64, 80]: WL items of the round
     cK = 96,        // [96, 112, 128]: vertices coloured in the round (stats)
-    cCol = 144,     // vertices coloured so far (host check)
+    cCol = 144,     // vertices coloured (written at the end, host check)
     cBar = 160,     // barrier arrivals (monotone)
     cAbort = 176,
     cErr = 192,     // [192..194] first trap: kind, round, vertex
@@ -89,8 +95,7 @@ struct CArgs {
     const uint32_t *ci;
     uint32_t *C;
     unsigned long long *cnt;  // (hi << 32) | lo
-    uint2 *Z;                 // first round at which the hi / lo side is free
-    uint32_t *sched;          // bit v: v has been scheduled (or coloured in round 0)
+    uint32_t *Zlo;            // round from which lo is free, when freed second (else kNever)
     Item *SL;
     Item *WL;
     unsigned long long *ctr;
@@ -165,7 +170,7 @@ constexpr int kStS = 4096, kStW = 4096, kStF = 4096;
 struct Stage {
     Item s[kStS];
     Item w[kStW];
-    uint32_t fresh[kStF];           // vertices this block scheduled in the round
+    uint2 fresh[kStF];              // (w, lo side?) this block scheduled in the round
     unsigned nf;
     unsigned n[2];
     unsigned colored;
@@ -237,10 +242,7 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
             }
         }
         st.nf = 0;
-        if (st.colored) {
-            atomicAdd(st.ccol, (unsigned long long)st.colored);
-            atomicAdd(&a.ctr[cCol], (unsigned long long)st.colored);
-        }
+        if (st.colored) atomicAdd(st.ccol, (unsigned long long)st.colored);
         st.colored = 0;
     }
     __syncthreads();
@@ -254,8 +256,7 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
 // row [rs, rs + len)) for the next round: short rows as one SL item, longer
 // rows as ceil(len / kSeg) WL items (expanded by the whole warp).
 __device__ __noinline__ void schedule_rows(const CArgs &a, bool pred, uint32_t w, int64_t rs,
-                                              int64_t len, bool first) {
-    const uint32_t ff = first ? kFirst : 0u;
+                                           int64_t len, uint32_t ff) {
     const bool shortrow = pred && len <= kShortMax;
     Item it;
     it.v = w;
@@ -269,6 +270,7 @@ __device__ __noinline__ void schedule_rows(const CArgs &a, bool pred, uint32_t w
         const uint32_t ww = __shfl_sync(kFull, w, src);
         const int64_t r0 = __shfl_sync(kFull, rs, src);
         const int64_t ln = __shfl_sync(kFull, len, src);
+        const uint32_t fs = __shfl_sync(kFull, ff, src);
         const uint32_t nseg = (uint32_t)((ln + kSeg - 1) / kSeg);
         for (uint32_t q0 = 0; q0 < nseg; q0 += 32) {
             const uint32_t q = q0 + lane_id();
@@ -276,7 +278,7 @@ __device__ __noinline__ void schedule_rows(const CArgs &a, bool pred, uint32_t w
             si.v = ww;
             const int64_t e0 = r0 + (int64_t)q * kSeg;
             si.e0 = e0;
-            si.lf = (uint32_t)min((int64_t)kSeg, r0 + ln - e0) | (q == 0 ? ff : 0u);
+            si.lf = (uint32_t)min((int64_t)kSeg, r0 + ln - e0) | (q == 0 ? fs : 0u);
             stage_append(a, q < nseg, si, 1);
         }
     }
@@ -284,10 +286,8 @@ __device__ __noinline__ void schedule_rows(const CArgs &a, bool pred, uint32_t w
 
 // Colour v in round k (its scheduled round): min (2k+1) if the lo side is
 // free at the start of round k, else max (2k) -- Alg.5 L37-42, R9.
-__device__ __forceinline__ void colour(const CArgs &a, uint32_t v, uint32_t k) {
-    const uint2 z = a.Z[v];
-    const bool lo_free = z.y <= k, hi_free = z.x <= k;
-    if (!lo_free && !hi_free) flag_error(a, 3, k, v);
+__device__ __forceinline__ void colour(const CArgs &a, uint32_t v, uint32_t lf, uint32_t k) {
+    const bool lo_free = (lf & kLoSide) || a.Zlo[v] <= k;
     a.C[v] = 2u * k + (lo_free ? 1u : 0u);
 }
 
@@ -322,10 +322,10 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
         if (w[q] != kNone) {
             ++nvis;
             const uint32_t side = hi[q] ? (uint32_t)(old[q] >> 32) : (uint32_t)old[q];
+            const uint32_t other = hi[q] ? (uint32_t)old[q] : (uint32_t)(old[q] >> 32);
             if (side == 1u) {
-                reinterpret_cast<uint32_t *>(a.Z + w[q])[hi[q] ? 0 : 1] = k + 1u;
-                const uint32_t bit = 1u << (w[q] & 31u);
-                fresh[q] = (atomicOr(&a.sched[w[q] >> 5], bit) & bit) == 0u;
+                if (other != 0u) fresh[q] = true;        // first side freed: schedule w
+                else if (!hi[q]) a.Zlo[w[q]] = k + 1u;   // lo freed second
             } else if (side == 0u) {
                 flag_error(a, 4, k, w[q]);  // count underflow: adjacency not symmetric
             }
@@ -340,7 +340,7 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
         ovf[q] = false;
         if (fresh[q]) {
             const unsigned pos = atomicAdd(&stage().nf, 1u);
-            if (pos < (unsigned)kStF) stage().fresh[pos] = w[q];
+            if (pos < (unsigned)kStF) stage().fresh[pos] = make_uint2(w[q], hi[q] ? 0u : kLoSide);
             else ovf[q] = true;
         }
     }
@@ -352,7 +352,7 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
                 rs = a.ro[w[q]];
                 re = a.ro[w[q] + 1];
             }
-            schedule_rows(a, ovf[q], w[q], rs, re - rs, true);
+            schedule_rows(a, ovf[q], w[q], rs, re - rs, kFirst | (hi[q] ? 0u : kLoSide));
         }
     }
 }
@@ -367,14 +367,14 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a) {
     for (unsigned base = wib * 32; base < nf; base += nwb * 32) {
         const unsigned idx = base + lane_id();
         const bool valid = idx < nf;
-        uint32_t w = 0;
+        uint2 f = make_uint2(0u, 0u);
         int64_t rs = 0, re = 0;
         if (valid) {
-            w = st.fresh[idx];
-            rs = a.ro[w];
-            re = a.ro[w + 1];
+            f = st.fresh[idx];
+            rs = a.ro[f.x];
+            re = a.ro[f.x + 1];
         }
-        schedule_rows(a, valid, w, rs, re - rs, true);
+        schedule_rows(a, valid, f.x, rs, re - rs, kFirst | f.y);
     }
 }
 
@@ -420,7 +420,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
         __syncthreads();
     }
     // ---------------------------------------------------- init = round 0
-    // lane per vertex, 32 consecutive vertices per warp (one sched word)
+    // lane per vertex: a zero count colours v in round 0 (min wins, R9)
     for (unsigned long long base = gwarp * 32; base < (unsigned long long)n; base += nwarps * 32) {
         const uint32_t v = (uint32_t)(base + lane);
         const bool valid = (int64_t)(base + lane) < n;
@@ -429,19 +429,16 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
         const bool zero = valid && (hi == 0u || lo == 0u);
         int64_t rs = 0, re = 0;
         if (valid) {
-            a.Z[v] = make_uint2(hi == 0u ? 0u : kNever, lo == 0u ? 0u : kNever);
-            a.C[v] = zero ? (lo == 0u ? 1u : 0u) : GC_UNC;  // round 0: min wins (R9)
+            a.Zlo[v] = kNever;
+            a.C[v] = zero ? (lo == 0u ? 1u : 0u) : GC_UNC;
             if (zero) {
                 rs = a.ro[v];
                 re = a.ro[v + 1];
             }
         }
         const unsigned word = __ballot_sync(kFull, zero);
-        if (lane == 0) {
-            a.sched[base >> 5] = word;
-            if (word) atomicAdd(&stage().colored, (unsigned)__popc(word));
-        }
-        schedule_rows(a, zero && re > rs, v, rs, re - rs, false);  // walked in round 0
+        if (lane == 0 && word) atomicAdd(&stage().colored, (unsigned)__popc(word));
+        schedule_rows(a, zero && re > rs, v, rs, re - rs, 0u);  // walked in round 0
     }
     stage_flush(a);
     if (!grid_barrier(a, 0)) return;
@@ -451,6 +448,11 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
         t0 = t;
     }
     // ------------------------------------------------------------ rounds
+    // work units of a round: WL items u < nw, then groups of 4 SL items; unit
+    // u goes to block u % G, warp (u / G) % wpb of it (round-robin over SMs)
+    const unsigned wpb = blockDim.x >> 5;
+    const unsigned long long u_first =
+        (unsigned long long)(threadIdx.x >> 5) * gridDim.x + blockIdx.x;
     unsigned long long sl0 = 0, wl0 = 0;  // where round k's items start
     int64_t rem = n;                      // gtid 0 only: uncoloured at the round start
     uint32_t last = 0;                    // last round with a colouring
@@ -481,33 +483,35 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
         const unsigned long long sl1 = sl0 + ns, wl1 = wl0 + nw;
         const unsigned long long t_round = PROF ? gtimer() : 0ull;
         set_targets(a, k, sl1, wl1);
-        // short rows: 4 per warp, 8 lanes each, 4 entries per lane
-        for (unsigned long long b = sl0 + gwarp * 4; b < sl1; b += nwarps * 4) {
-            const unsigned long long idx = b + (lane >> 3);
-            uint32_t v = kNone, len = 0, pv = 0;
-            int64_t e0 = 0;
-            if (idx < sl1) {
-                const Item it = a.SL[idx];
-                v = it.v;
-                len = it.lf & ~kFirst;
-                e0 = it.e0;
-                pv = weight_mix(v ^ a.key);
-                if ((it.lf & kFirst) && (lane & 7u) == 0u) {
-                    colour(a, v, k);
+        const unsigned long long units = nw + (ns + 3) / 4;
+        for (unsigned long long u = u_first; u < units; u += nwarps) {
+            if (u < nw) {
+                // longer rows: one <= kSeg-entry item per warp
+                const Item it = a.WL[wl0 + u];
+                const uint32_t pv = weight_mix(it.v ^ a.key);
+                if ((it.lf & kFirst) && lane == 0) {
+                    colour(a, it.v, it.lf, k);
                     atomicAdd(&stage().colored, 1u);
                 }
+                walk<kSeg / 32>(a, it.v, pv, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k, nvis);
+            } else {
+                // short rows: 4 per warp, 8 lanes each, 4 entries per lane
+                const unsigned long long idx = sl0 + 4 * (u - nw) + (lane >> 3);
+                uint32_t v = kNone, len = 0, pv = 0;
+                int64_t e0 = 0;
+                if (idx < sl1) {
+                    const Item it = a.SL[idx];
+                    v = it.v;
+                    len = it.lf & kLenMask;
+                    e0 = it.e0;
+                    pv = weight_mix(v ^ a.key);
+                    if ((it.lf & kFirst) && (lane & 7u) == 0u) {
+                        colour(a, v, it.lf, k);
+                        atomicAdd(&stage().colored, 1u);
+                    }
+                }
+                walk<4>(a, v, pv, e0 + (lane & 7u), e0 + len, 8, k, nvis);
             }
-            walk<4>(a, v, pv, e0 + (lane & 7u), e0 + len, 8, k, nvis);
-        }
-        // longer rows: one <= kSeg-entry item per warp
-        for (unsigned long long i = wl0 + gwarp; i < wl1; i += nwarps) {
-            const Item it = a.WL[i];
-            const uint32_t pv = weight_mix(it.v ^ a.key);
-            if ((it.lf & kFirst) && lane == 0) {
-                colour(a, it.v, k);
-                atomicAdd(&stage().colored, 1u);
-            }
-            walk<kSeg / 32>(a, it.v, pv, it.e0 + lane, it.e0 + (it.lf & ~kFirst), 32, k, nvis);
         }
         sl0 = sl1;
         wl0 = wl1;
@@ -527,9 +531,11 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
             t0 = t;
         }
     }
+    (void)wpb;
     if (gtid == 0) {
         a.ctr[cRounds] = n > 0 ? last + 1 : 0;
         a.ctr[cIters] = k;
+        a.ctr[cCol] = (unsigned long long)(n - rem);
         if (PROF) a.ctr[cPhaseNs + 1] = t_rounds;
     }
     if (PROF) {
@@ -655,8 +661,7 @@ int ensure_count_scratch(gc_graph *g) {
     const size_t nn = (size_t)std::max<int64_t>(g->n, 1);
     if (s.cnt) return GC_OK;
     GC_CUDA_TRY(dmalloc(&s.cnt, nn * 8));
-    GC_CUDA_TRY(dmalloc(&s.Z, nn * 8));
-    GC_CUDA_TRY(dmalloc(&s.sched, ((nn + 31) / 32) * 4));
+    GC_CUDA_TRY(dmalloc(&s.Z, nn * 4));
     s.sl_cap = (int64_t)nn;
     s.wl_cap = (int64_t)nn + g->nnz / kSeg + 1;
     GC_CUDA_TRY(dmalloc(&s.SL, (size_t)s.sl_cap * sizeof(Item)));
@@ -704,8 +709,7 @@ int run_count_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     a.ci = g->ci;
     a.C = s.C;
     a.cnt = s.cnt;
-    a.Z = reinterpret_cast<uint2 *>(s.Z);
-    a.sched = s.sched;
+    a.Zlo = s.Z;
     a.SL = reinterpret_cast<Item *>(s.SL);
     a.WL = reinterpret_cast<Item *>(s.WL);
     a.ctr = s.cctr;

@@ -63,8 +63,7 @@ struct Scratch {
     int64_t *host_pinned = nullptr;  // pinned readback area
     // COUNT mode (gc_count.cu)
     unsigned long long *cnt = nullptr;   // (hi << 32) | lo uncoloured-neighbour counts
-    uint32_t *Z = nullptr;               // uint2 per vertex: round from which hi / lo is free
-    uint32_t *sched = nullptr;           // scheduled bit per vertex
+    uint32_t *Z = nullptr;               // Zlo: round from which lo is free (freed second)
     void *SL = nullptr;                  // short-row items (16 B)
     void *WL = nullptr;                  // long-row segment items (16 B)
     uint32_t *hubs = nullptr;            // k_count: rows counted by blocks
