@@ -132,6 +132,17 @@ __device__ __forceinline__ unsigned long long atom_add_release(unsigned long lon
     return v;
 }
 
+// 64-bit add on GLOBAL memory.  atomicAdd through a generic pointer (CArgs
+// members) compiles to ATOM.E + a shared-memory CAS fallback branch, which
+// serialises a lane's atomics (each waits for the previous one's predicate);
+// the global form lets all Q atomics of a lane be in flight together.
+__device__ __forceinline__ unsigned long long atom_add_global(unsigned long long *p,
+                                                              unsigned long long x) {
+    unsigned long long old;
+    asm volatile("atom.global.add.u64 %0, [%1], %2;" : "=l"(old) : "l"(p), "l"(x));
+    return old;
+}
+
 // Grid barrier (cooperative launch: every block is resident): monotone
 // arrival counter, release arrival, acquire spin (which also invalidates the
 // SM's L1, so the next phase sees what other SMs wrote).  A wait beyond 4 s
@@ -208,7 +219,7 @@ __device__ __forceinline__ void stage_append(const CArgs &a, bool pred, const It
     if (sm) {
         const unsigned sl = __ffs(sm) - 1;
         unsigned long long gb = 0;
-        if (lane == sl) gb = atomicAdd(st.cnext[li], (unsigned long long)__popc(sm));
+        if (lane == sl) gb = atom_add_global(st.cnext[li], (unsigned long long)__popc(sm));
         gb = __shfl_sync(kFull, gb, sl);
         if (spill) {
             const unsigned long long at = st.nbase[li] + gb + __popc(sm & ((1u << lane) - 1u));
@@ -234,7 +245,7 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
         for (int i = 0; i < 2; ++i) {
             const unsigned c = min(st.n[i], (unsigned)(i == 0 ? kStS : kStW));
             st.n[i] = c;
-            st.base[i] = c ? st.nbase[i] + atomicAdd(st.cnext[i], (unsigned long long)c) : 0ull;
+            st.base[i] = c ? st.nbase[i] + atom_add_global(st.cnext[i], (unsigned long long)c) : 0ull;
             const unsigned long long capg = i == 0 ? a.sl_cap : a.wl_cap;
             if (c && st.base[i] + c > capg) {
                 flag_error(a, 2, 0, (unsigned)i);
@@ -242,7 +253,7 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
             }
         }
         st.nf = 0;
-        if (st.colored) atomicAdd(st.ccol, (unsigned long long)st.colored);
+        if (st.colored) atom_add_global(st.ccol, (unsigned long long)st.colored);
         st.colored = 0;
     }
     __syncthreads();
@@ -250,13 +261,15 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
     for (unsigned i = threadIdx.x; i < st.n[1]; i += blockDim.x) a.WL[st.base[1] + i] = st.w[i];
     __syncthreads();
     if (threadIdx.x < 2) st.n[threadIdx.x] = 0;
+    if (prs && threadIdx.x == 0)
+        atomicMax(reinterpret_cast<unsigned long long *>(prs + 8), gtimer() - t_round);
 }
 
 // Whole warp converged: schedule the rows of the lanes with `pred` (vertex w,
 // row [rs, rs + len)) for the next round: short rows as one SL item, longer
 // rows as ceil(len / kSeg) WL items (expanded by the whole warp).
-__device__ __noinline__ void schedule_rows(const CArgs &a, bool pred, uint32_t w, int64_t rs,
-                                           int64_t len, uint32_t ff) {
+__device__ __forceinline__ void schedule_rows(const CArgs &a, bool pred, uint32_t w, int64_t rs,
+                                              int64_t len, uint32_t ff) {
     const bool shortrow = pred && len <= kShortMax;
     Item it;
     it.v = w;
@@ -282,6 +295,13 @@ __device__ __noinline__ void schedule_rows(const CArgs &a, bool pred, uint32_t w
             stage_append(a, q < nseg, si, 1);
         }
     }
+}
+
+// Out-of-line copy for the rare paths inside the unrolled walk (overflowing
+// fresh list): keeps walk's code and registers small.
+__device__ __noinline__ void schedule_rows_slow(const CArgs &a, bool pred, uint32_t w, int64_t rs,
+                                                int64_t len, uint32_t ff) {
+    schedule_rows(a, pred, w, rs, len, ff);
 }
 
 // Colour v in round k (its scheduled round): min (2k+1) if the lo side is
@@ -312,7 +332,7 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
         old[q] = 0;
         if (w[q] != kNone) {
             hi[q] = pv > weight_mix(w[q] ^ a.key);  // v is a larger neighbour of w
-            old[q] = atomicAdd(&a.cnt[w[q]], hi[q] ? kDecHi : kDecLo);
+            old[q] = atom_add_global(a.cnt + w[q], hi[q] ? kDecHi : kDecLo);
         }
     }
     bool fresh[Q];
@@ -352,16 +372,22 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
                 rs = a.ro[w[q]];
                 re = a.ro[w[q] + 1];
             }
-            schedule_rows(a, ovf[q], w[q], rs, re - rs, kFirst | (hi[q] ? 0u : kLoSide));
+            schedule_rows_slow(a, ovf[q], w[q], rs, re - rs, kFirst | (hi[q] ? 0u : kLoSide));
         }
     }
 }
 
 // Whole block, end of a round: stage the items of the vertices on the fresh
 // list (all their row offsets are fetched in one dependent step).
-__device__ __forceinline__ void schedule_fresh(const CArgs &a) {
+__device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nullptr,
+                                               unsigned long long t_round = 0) {
     Stage &st = stage();
     __syncthreads();
+    if (prs && threadIdx.x == 0) {  // PROF: this block's units are done
+        const unsigned long long dt = gtimer() - t_round;
+        atomicMax(reinterpret_cast<unsigned long long *>(prs + 7), dt);
+        atomicMax(reinterpret_cast<unsigned long long *>(prs + 9), ~dt);  // min via ~
+    }
     const unsigned nf = min(st.nf, (unsigned)kStF);
     const unsigned wib = threadIdx.x >> 5, nwb = blockDim.x >> 5;
     for (unsigned base = wib * 32; base < nf; base += nwb * 32) {
@@ -458,6 +484,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
     uint32_t last = 0;                    // last round with a colouring
     uint32_t k = 0;
     for (;; ++k) {
+        const unsigned long long t_round = PROF ? gtimer() : 0ull;
         const int cur = (int)(k % 3);
         const unsigned long long ns = __ldcg(&a.ctr[cS + 16 * cur]), nw = __ldcg(&a.ctr[cW + 16 * cur]);
         if (gtid == 0) {
@@ -481,10 +508,13 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
             a.rstat[16 * k + 1] = (int64_t)nw;
         }
         const unsigned long long sl1 = sl0 + ns, wl1 = wl0 + nw;
-        const unsigned long long t_round = PROF ? gtimer() : 0ull;
         set_targets(a, k, sl1, wl1);
+        int64_t *prs = (PROF && (int64_t)k < a.nk_cap) ? a.rstat + 16 * k : nullptr;
+        if (prs && threadIdx.x == 0)
+            atomicMax(reinterpret_cast<unsigned long long *>(prs + 6), gtimer() - t_round);
         const unsigned long long units = nw + (ns + 3) / 4;
         for (unsigned long long u = u_first; u < units; u += nwarps) {
+            const long long c_unit = PROF ? clock64() : 0;
             if (u < nw) {
                 // longer rows: one <= kSeg-entry item per warp
                 const Item it = a.WL[wl0 + u];
@@ -512,6 +542,9 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
                 }
                 walk<4>(a, v, pv, e0 + (lane & 7u), e0 + len, 8, k, nvis);
             }
+            if (prs && lane == 0)
+                atomicMax(reinterpret_cast<unsigned long long *>(prs + 10),
+                          (unsigned long long)(clock64() - c_unit));
         }
         sl0 = sl1;
         wl0 = wl1;
@@ -521,8 +554,8 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
             nvis_tot += nvis;
             nvis = 0;
         }
-        schedule_fresh(a);
-        stage_flush(a, (PROF && (int64_t)k < a.nk_cap) ? a.rstat + 16 * k : nullptr, t_round);
+        schedule_fresh(a, prs, t_round);
+        stage_flush(a, prs, t_round);
         if (!grid_barrier(a, k)) return;
         if (PROF && gtid == 0) {
             const unsigned long long t = gtimer();

@@ -41,7 +41,13 @@ def main():
     for r in range(R):
         rs = st.round_stats[16 * r: 16 * r + 16]
         # persistent kernel: per-phase times (ns) are in the round record
-        if mode == gcb.MODE_COUNT:  # [SL items, WL items, entries, coloured, round ns, max block ns]
+        if mode == gcb.MODE_COUNT:
+            # [SL items, WL items, entries, coloured, round ns, max ns to flush start,
+            #  max ns to targets set, max ns units done, max ns flush done,
+            #  min ns units done (stored as ~ns), max cycles of one unit]
+            rs = list(rs)
+            if rs[9] < 0:
+                rs[9] = -rs[9] - 1
             t = [rs[4] / 1e3]
         elif mode == gcb.MODE_EVENT:
             t = [x / 1e3 for x in rs[4:7]]
