@@ -343,6 +343,9 @@ static void free_scratch(Scratch &s) {
     dfree(s.bitmap);
     dfree(s.hist);
     dfree(s.cnt);
+    dfree(s.cnt32);
+    dfree(s.big);
+    dfree(s.big32);
     dfree(s.Z);
     dfree(s.SL);
     dfree(s.WL);

@@ -41,6 +41,10 @@
 
 #include "gc_internal.cuh"
 
+#ifndef GC_PACKED
+#define GC_PACKED 0  // 1: 32-bit (hi << 16 | lo) round counts (measured 0.8 ms slower on R-MAT s24)
+#endif
+
 namespace gc {
 
 int ensure_nk(gc_graph *g, int64_t need);
@@ -59,6 +63,15 @@ constexpr uint32_t kFirst = 0x80000000u;   // item flag: colour v in this round
 constexpr uint32_t kLoSide = 0x40000000u;  // item flag: scheduled by its lo side (min colour)
 constexpr uint32_t kLenMask = 0x3FFFFFFFu;
 constexpr unsigned long long kDecHi = 0ull - (1ull << 32);
+// Packed counts: the rounds decrement a 32-bit word (hi << 16 | lo) per vertex
+// -- half the footprint of 64-bit words, so the round's burst of random
+// atomics mostly hits L2 (tools/microbench_atomics.cu: a 205k-atomic burst
+// takes 1.6 us on a 67 MB array, 3.6 us on 134 MB, whatever the width).
+// Vertices of degree > kPackMax ("big") keep 64-bit words; they are few and
+// are found through a hash set in shared memory (no extra global access).
+constexpr int64_t kPackMax = 65535;
+constexpr int kHTab = 4096;                // shared hash slots (big vertices <= kHTab / 2)
+constexpr uint32_t kDec32Hi = 0u - (1u << 16);
 constexpr unsigned long long kDecLo = ~0ull;
 
 __device__ __forceinline__ unsigned lane_id() { return threadIdx.x & 31u; }
@@ -94,7 +107,12 @@ struct CArgs {
     const int64_t *ro;
     const uint32_t *ci;
     uint32_t *C;
-    unsigned long long *cnt;  // (hi << 32) | lo
+    unsigned long long *cnt;  // (hi << 32) | lo from the counting kernels (read by init)
+    uint32_t *cnt32;          // the rounds' counts: (hi << 16) | lo per vertex, or ...
+    uint32_t *big32;          // ... for big vertices, [2 s] = hi, [2 s + 1] = lo, [2 kHTab + s] =
+                              // "scheduled" flag, s = the vertex's slot in the shared hash set
+    const uint32_t *big;      // big vertices (degree > kPackMax)
+    int nbig;
     uint32_t *Zlo;            // round from which lo is free, when freed second (else kNever)
     Item *SL;
     Item *WL;
@@ -143,6 +161,24 @@ __device__ __forceinline__ unsigned long long atom_add_global(unsigned long long
     return old;
 }
 
+// fire-and-forget PROF counters (no wait for a result)
+__device__ __forceinline__ void red_max(int64_t *p, unsigned long long x) {
+    asm volatile("red.global.max.u64 [%0], %1;" ::"l"(p), "l"(x) : "memory");
+}
+__device__ __forceinline__ void red_add(int64_t *p, unsigned long long x) {
+    asm volatile("red.global.add.u64 [%0], %1;" ::"l"(p), "l"(x) : "memory");
+}
+__device__ __forceinline__ uint32_t atom_or_global(uint32_t *p, uint32_t x) {
+    uint32_t old;
+    asm volatile("atom.global.or.b32 %0, [%1], %2;" : "=r"(old) : "l"(p), "r"(x));
+    return old;
+}
+__device__ __forceinline__ uint32_t atom_add_global32(uint32_t *p, uint32_t x) {
+    uint32_t old;
+    asm volatile("atom.global.add.u32 %0, [%1], %2;" : "=r"(old) : "l"(p), "r"(x));
+    return old;
+}
+
 // Grid barrier (cooperative launch: every block is resident): monotone
 // arrival counter, release arrival, acquire spin (which also invalidates the
 // SM's L1, so the next phase sees what other SMs wrote).  A wait beyond 4 s
@@ -177,15 +213,22 @@ __device__ __forceinline__ bool grid_barrier(const CArgs &a, uint32_t k) {
 }
 
 // ---------------------------------------------------------------- staging
-constexpr int kStS = 4096, kStW = 4096, kStF = 4096;
+constexpr int kStS = 4096, kStW = 4096, kStF = 4096, kLongMax = 512;
 struct Stage {
     Item s[kStS];
     Item w[kStW];
     uint2 fresh[kStF];              // (w, lo side?) this block scheduled in the round
+    uint32_t htab[kHTab];           // hash set of the big vertices (kNone = empty)
+    struct Long {                   // schedule_fresh: a long row to expand
+        int64_t rs, dst;            // row start; first item slot (>= 0 staged, < 0: ~global)
+        uint32_t w, len, flags, pad;
+    } lng[kLongMax];
+    unsigned nlong;
     unsigned nf;
     unsigned n[2];
     unsigned colored;
     unsigned vis;                   // PROF: entries walked by this block in the round
+    unsigned long long t_fs;        // PROF: when this block's fresh step started
     unsigned long long base[2];
     // append targets of the current round (set by thread 0 at the round top)
     unsigned long long *cnext[2];   // item-count slots of the next round
@@ -197,6 +240,17 @@ constexpr size_t kStageBytes = sizeof(Stage);
 __device__ __forceinline__ Stage &stage() {
     extern __shared__ __align__(16) unsigned char smem_raw[];
     return *reinterpret_cast<Stage *>(smem_raw);
+}
+
+__device__ __forceinline__ unsigned hslot(uint32_t v) { return (v * 2654435761u) >> 20; }  // 12 bits
+// slot of v in the block's hash set of big vertices, or -1
+__device__ __forceinline__ int big_slot(uint32_t v) {
+    const uint32_t *t = stage().htab;
+    for (unsigned h = hslot(v);; h = (h + 1) & (kHTab - 1)) {
+        const uint32_t x = t[h];
+        if (x == v) return (int)h;
+        if (x == kNone) return -1;
+    }
 }
 
 // Whole warp converged: lanes with `pred` append `val` to staged list li;
@@ -237,8 +291,11 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
     Stage &st = stage();
     __syncthreads();
     if (prs && threadIdx.x == 0) {
-        atomicAdd(reinterpret_cast<unsigned long long *>(prs + 2), (unsigned long long)st.vis);
-        atomicMax(reinterpret_cast<unsigned long long *>(prs + 5), gtimer() - t_round);
+        const unsigned long long fdt = gtimer() - st.t_fs;  // this block's fresh step
+        red_add(prs + 11, fdt);
+        red_max(prs + 12, fdt);
+        red_add(prs + 2, (unsigned long long)st.vis);
+        red_max(prs + 5, gtimer() - t_round);
         st.vis = 0;
     }
     if (threadIdx.x == 0) {
@@ -262,7 +319,7 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
     __syncthreads();
     if (threadIdx.x < 2) st.n[threadIdx.x] = 0;
     if (prs && threadIdx.x == 0)
-        atomicMax(reinterpret_cast<unsigned long long *>(prs + 8), gtimer() - t_round);
+        red_max(prs + 8, gtimer() - t_round);
 }
 
 // Whole warp converged: schedule the rows of the lanes with `pred` (vertex w,
@@ -275,6 +332,10 @@ __device__ __forceinline__ void schedule_rows(const CArgs &a, bool pred, uint32_
     it.v = w;
     it.lf = (uint32_t)len | ff;
     it.e0 = rs;
+    if (shortrow && len > 0) {  // the row walked next round: HBM -> L2 now (<= 2 lines)
+        asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ci + rs));
+        asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ci + rs + len - 1));
+    }
     stage_append(a, shortrow, it, 0);
     unsigned lm = __ballot_sync(kFull, pred && !shortrow);
     while (lm) {
@@ -324,16 +385,29 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
         const int64_t eq = e + (int64_t)q * stride;
         w[q] = (v != kNone && eq < end) ? __ldcs(a.ci + eq) : kNone;
     }
+    // One 32-bit atomic per entry, address and value chosen without a branch
+    // (a branch around each atomic made the compiler wait for every result).
+#if GC_PACKED
+    uint32_t old[Q];
+#else
     unsigned long long old[Q];
+#endif
     bool hi[Q];
+    int slot[Q];
 #pragma unroll
     for (int q = 0; q < Q; ++q) {
-        hi[q] = false;
-        old[q] = 0;
-        if (w[q] != kNone) {
-            hi[q] = pv > weight_mix(w[q] ^ a.key);  // v is a larger neighbour of w
-            old[q] = atom_add_global(a.cnt + w[q], hi[q] ? kDecHi : kDecLo);
-        }
+        const bool live = w[q] != kNone;
+        const uint32_t wq = live ? w[q] : 0u;
+        hi[q] = live && pv > weight_mix(wq ^ a.key);  // v is a larger neighbour of w
+#if GC_PACKED
+        slot[q] = (live && a.nbig > 0) ? big_slot(wq) : -1;
+        uint32_t *adr = slot[q] >= 0 ? a.big32 + 2 * slot[q] + (hi[q] ? 0 : 1) : a.cnt32 + wq;
+        const uint32_t dec = (slot[q] < 0 && hi[q]) ? kDec32Hi : 0xFFFFFFFFu;
+        old[q] = live ? atom_add_global32(adr, dec) : 2u;
+#else
+        slot[q] = -1;
+        old[q] = live ? atom_add_global(a.cnt + wq, hi[q] ? kDecHi : kDecLo) : 2ull;
+#endif
     }
     bool fresh[Q];
 #pragma unroll
@@ -341,8 +415,18 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
         fresh[q] = false;
         if (w[q] != kNone) {
             ++nvis;
-            const uint32_t side = hi[q] ? (uint32_t)(old[q] >> 32) : (uint32_t)old[q];
-            const uint32_t other = hi[q] ? (uint32_t)old[q] : (uint32_t)(old[q] >> 32);
+            uint32_t side, other;
+            if (!GC_PACKED) {
+                side = hi[q] ? (uint32_t)(old[q] >> 32) : (uint32_t)old[q];
+                other = hi[q] ? (uint32_t)old[q] : (uint32_t)(old[q] >> 32);
+            } else if (slot[q] < 0) {
+                side = hi[q] ? (uint32_t)old[q] >> 16 : (uint32_t)old[q] & 0xFFFFu;
+                other = hi[q] ? (uint32_t)old[q] & 0xFFFFu : (uint32_t)old[q] >> 16;
+            } else {  // big vertex: a side reaching zero claims the flag (rare)
+                side = old[q];
+                other = 1u;
+                if (side == 1u) other = atom_or_global(a.big32 + 2 * kHTab + slot[q], 1u) ? 0u : 1u;
+            }
             if (side == 1u) {
                 if (other != 0u) fresh[q] = true;        // first side freed: schedule w
                 else if (!hi[q]) a.Zlo[w[q]] = k + 1u;   // lo freed second
@@ -359,6 +443,9 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
     for (int q = 0; q < Q; ++q) {
         ovf[q] = false;
         if (fresh[q]) {
+            // its row offsets are loaded at the end of the round: start the
+            // HBM -> L2 transfer now
+            asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ro + w[q]));
             const unsigned pos = atomicAdd(&stage().nf, 1u);
             if (pos < (unsigned)kStF) stage().fresh[pos] = make_uint2(w[q], hi[q] ? 0u : kLoSide);
             else ovf[q] = true;
@@ -378,29 +465,88 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
 }
 
 // Whole block, end of a round: stage the items of the vertices on the fresh
-// list (all their row offsets are fetched in one dependent step).
+// list -- one THREAD per fresh vertex (row offsets in one dependent step),
+// then the segments of all long rows written by the whole block.  An SL
+// overflow, a long row that does not fit the staged WL buffer and a long-row
+// list overflow go straight to the global lists (rare).
 __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nullptr,
                                                unsigned long long t_round = 0) {
     Stage &st = stage();
+    if (threadIdx.x == 0) st.nlong = 0;
     __syncthreads();
     if (prs && threadIdx.x == 0) {  // PROF: this block's units are done
         const unsigned long long dt = gtimer() - t_round;
-        atomicMax(reinterpret_cast<unsigned long long *>(prs + 7), dt);
-        atomicMax(reinterpret_cast<unsigned long long *>(prs + 9), ~dt);  // min via ~
+        red_max(prs + 7, dt);
+        red_max(prs + 9, ~dt);  // min via ~
+        red_max(prs + 13, (unsigned long long)st.nf);
+        st.t_fs = gtimer();
     }
     const unsigned nf = min(st.nf, (unsigned)kStF);
-    const unsigned wib = threadIdx.x >> 5, nwb = blockDim.x >> 5;
-    for (unsigned base = wib * 32; base < nf; base += nwb * 32) {
-        const unsigned idx = base + lane_id();
-        const bool valid = idx < nf;
-        uint2 f = make_uint2(0u, 0u);
-        int64_t rs = 0, re = 0;
-        if (valid) {
-            f = st.fresh[idx];
-            rs = a.ro[f.x];
-            re = a.ro[f.x + 1];
+    for (unsigned t = threadIdx.x; t < nf; t += blockDim.x) {
+        const uint2 f = st.fresh[t];
+        const int64_t rs = a.ro[f.x], re = a.ro[f.x + 1];
+        const int64_t len = re - rs;
+        const uint32_t fl = kFirst | f.y;
+        if (len <= kShortMax) {
+            Item it;
+            it.v = f.x;
+            it.lf = (uint32_t)len | fl;
+            it.e0 = rs;
+            if (len > 0) {  // the row walked next round: HBM -> L2 now (<= 2 lines)
+                asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ci + rs));
+                asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ci + re - 1));
+            }
+            const unsigned pos = atomicAdd(&st.n[0], 1u);
+            if (pos < (unsigned)kStS) {
+                st.s[pos] = it;
+            } else {
+                const unsigned long long at = st.nbase[0] + atom_add_global(st.cnext[0], 1ull);
+                if (at < a.sl_cap) a.SL[at] = it;
+                else flag_error(a, 1, 0, f.x);
+            }
+        } else {
+            const uint32_t nseg = (uint32_t)((len + kSeg - 1) / kSeg);
+            const unsigned sb = atomicAdd(&st.n[1], nseg);
+            int64_t dst;
+            if (sb + nseg <= (unsigned)kStW) {
+                dst = (int64_t)sb;
+            } else {
+                // does not fit: global slots; staged slots [sb, kStW) become holes
+                for (unsigned h = sb; h < (unsigned)kStW && h < sb + nseg; ++h) st.w[h].v = kNone;
+                dst = ~(int64_t)(st.nbase[1] + atom_add_global(st.cnext[1], (unsigned long long)nseg));
+            }
+            const unsigned li = atomicAdd(&st.nlong, 1u);
+            if (li < (unsigned)kLongMax) {
+                st.lng[li].rs = rs;
+                st.lng[li].dst = dst;
+                st.lng[li].w = f.x;
+                st.lng[li].len = (uint32_t)len;
+                st.lng[li].flags = fl;
+            } else {  // long-row list full: this thread writes the segments itself
+                for (uint32_t q = 0; q < nseg; ++q) {
+                    Item si;
+                    si.v = f.x;
+                    si.e0 = rs + (int64_t)q * kSeg;
+                    si.lf = (uint32_t)min((int64_t)kSeg, len - (int64_t)q * kSeg) | (q == 0 ? fl : 0u);
+                    if (dst >= 0) st.w[dst + q] = si;
+                    else a.WL[~dst + q] = si;
+                }
+            }
         }
-        schedule_rows(a, valid, f.x, rs, re - rs, kFirst | f.y);
+    }
+    __syncthreads();
+    const unsigned nl = min(st.nlong, (unsigned)kLongMax);
+    for (unsigned r = 0; r < nl; ++r) {
+        const Stage::Long L = st.lng[r];
+        const uint32_t nseg = (L.len + kSeg - 1) / kSeg;
+        for (uint32_t q = threadIdx.x; q < nseg; q += blockDim.x) {
+            Item si;
+            si.v = L.w;
+            si.e0 = L.rs + (int64_t)q * kSeg;
+            si.lf = (uint32_t)min((int64_t)kSeg, (int64_t)L.len - (int64_t)q * kSeg) | (q == 0 ? L.flags : 0u);
+            if (L.dst >= 0) st.w[L.dst + q] = si;
+            else a.WL[~L.dst + q] = si;
+        }
     }
 }
 
@@ -435,6 +581,16 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
         if (threadIdx.x == 0) st.colored = 0;
         if (threadIdx.x == 0) st.vis = 0;
         if (threadIdx.x == 0) st.nf = 0;
+        for (int i = threadIdx.x; i < kHTab; i += blockDim.x) st.htab[i] = kNone;
+        __syncthreads();
+        if (threadIdx.x == 0) {
+            for (int i = 0; i < a.nbig; ++i) {
+                const uint32_t v = a.big[i];
+                unsigned h = hslot(v);
+                while (st.htab[h] != kNone) h = (h + 1) & (kHTab - 1);
+                st.htab[h] = v;
+            }
+        }
         // init appends round 0's items to slot 0 at position 0; its colourings
         // count for round 0 (so the "next round" targets are round 0's here)
         if (threadIdx.x == 0) {
@@ -455,6 +611,15 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
         const bool zero = valid && (hi == 0u || lo == 0u);
         int64_t rs = 0, re = 0;
         if (valid) {
+            const int sl = (GC_PACKED && a.nbig > 0) ? big_slot(v) : -1;
+            if (!GC_PACKED) {
+            } else if (sl < 0) {
+                a.cnt32[v] = (hi << 16) | lo;  // deg <= kPackMax
+            } else {
+                a.big32[2 * sl] = hi;
+                a.big32[2 * sl + 1] = lo;
+                a.big32[2 * kHTab + sl] = (hi == 0u || lo == 0u) ? 1u : 0u;
+            }
             a.Zlo[v] = kNever;
             a.C[v] = zero ? (lo == 0u ? 1u : 0u) : GC_UNC;
             if (zero) {
@@ -511,19 +676,41 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
         set_targets(a, k, sl1, wl1);
         int64_t *prs = (PROF && (int64_t)k < a.nk_cap) ? a.rstat + 16 * k : nullptr;
         if (prs && threadIdx.x == 0)
-            atomicMax(reinterpret_cast<unsigned long long *>(prs + 6), gtimer() - t_round);
-        const unsigned long long units = nw + (ns + 3) / 4;
+            red_max(prs + 6, gtimer() - t_round);
+        // a large SL list (round 0: millions of mostly 1-4-entry rows) is
+        // walked one row per LANE, so a warp has 32 rows in flight, not 4
+        const bool lane_rows = ns > 16ull * nwarps;
+        const unsigned long long units = nw + (lane_rows ? (ns + 31) / 32 : (ns + 3) / 4);
         for (unsigned long long u = u_first; u < units; u += nwarps) {
             const long long c_unit = PROF ? clock64() : 0;
             if (u < nw) {
                 // longer rows: one <= kSeg-entry item per warp
-                const Item it = a.WL[wl0 + u];
+                Item it = a.WL[wl0 + u];
+                if (it.v == kNone) it.lf = 0;  // hole left by schedule_fresh
                 const uint32_t pv = weight_mix(it.v ^ a.key);
                 if ((it.lf & kFirst) && lane == 0) {
                     colour(a, it.v, it.lf, k);
                     atomicAdd(&stage().colored, 1u);
                 }
                 walk<kSeg / 32>(a, it.v, pv, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k, nvis);
+            } else if (lane_rows) {
+                // short rows: one per lane, 4 entries per step
+                const unsigned long long idx = sl0 + 32 * (u - nw) + lane;
+                uint32_t v = kNone, len = 0, pv = 0;
+                int64_t e0 = 0;
+                if (idx < sl1) {
+                    const Item it = a.SL[idx];
+                    v = it.v;
+                    len = it.lf & kLenMask;
+                    e0 = it.e0;
+                    pv = weight_mix(v ^ a.key);
+                    if (it.lf & kFirst) {
+                        colour(a, v, it.lf, k);
+                        atomicAdd(&stage().colored, 1u);
+                    }
+                }
+                for (uint32_t j = 0; __any_sync(kFull, j < len); j += 4)
+                    walk<4>(a, j < len ? v : kNone, pv, e0 + j, e0 + len, 1, k, nvis);
             } else {
                 // short rows: 4 per warp, 8 lanes each, 4 entries per lane
                 const unsigned long long idx = sl0 + 4 * (u - nw) + (lane >> 3);
@@ -543,8 +730,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
                 walk<4>(a, v, pv, e0 + (lane & 7u), e0 + len, 8, k, nvis);
             }
             if (prs && lane == 0)
-                atomicMax(reinterpret_cast<unsigned long long *>(prs + 10),
-                          (unsigned long long)(clock64() - c_unit));
+                red_max(prs + 10, (unsigned long long)(clock64() - c_unit));
         }
         sl0 = sl1;
         wl0 = wl1;
@@ -679,9 +865,44 @@ int launch(gc_graph *g, CArgs &a, int *blocks_out) {
         return GC_ERR_CUDA;
     }
     const int blocks = per_sm * g->sm_count;
-    void *args[] = {&a};
-    GC_CUDA_TRY(cudaLaunchCooperativeKernel((void *)k_count_persistent<PROF>, blocks, kThreads, args,
-                                            kStageBytes, g->stream));
+    // L2 persistence for the count words (every round's decrements are a
+    // burst of random 8-byte atomics; a burst that misses L2 is several times
+    // slower, tools/microbench_atomics.cu).  Per-launch attribute: no stream
+    // or device state is changed except the persisting-L2 carve-out.
+    cudaLaunchAttribute attrs[2];
+    int na = 0;
+    attrs[na].id = cudaLaunchAttributeCooperative;
+    attrs[na].val.cooperative = 1;
+    ++na;
+    int dev = 0, max_persist = 0, max_window = 0;
+    cudaGetDevice(&dev);
+    cudaDeviceGetAttribute(&max_persist, cudaDevAttrMaxPersistingL2CacheSize, dev);
+    cudaDeviceGetAttribute(&max_window, cudaDevAttrMaxAccessPolicyWindowSize, dev);
+    const char *env = std::getenv("GC_L2_PERSIST");
+    // opt-in only: measured slower on R-MAT s24 (40.6 vs 35.7 ms)
+    const bool persist = max_persist > 0 && max_window > 0 && env && env[0] == '1';
+    if (persist) {
+        size_t cur = 0;
+        cudaDeviceGetLimit(&cur, cudaLimitPersistingL2CacheSize);
+        if (cur < (size_t)max_persist) cudaDeviceSetLimit(cudaLimitPersistingL2CacheSize, (size_t)max_persist);
+        const size_t bytes = std::min<size_t>((size_t)a.n * 8, (size_t)max_window);
+        attrs[na].id = cudaLaunchAttributeAccessPolicyWindow;
+        attrs[na].val.accessPolicyWindow.base_ptr = a.cnt;
+        attrs[na].val.accessPolicyWindow.num_bytes = bytes;
+        attrs[na].val.accessPolicyWindow.hitRatio =
+            (float)std::min(1.0, (double)max_persist / (double)std::max<size_t>(bytes, 1));
+        attrs[na].val.accessPolicyWindow.hitProp = cudaAccessPropertyPersisting;
+        attrs[na].val.accessPolicyWindow.missProp = cudaAccessPropertyStreaming;
+        ++na;
+    }
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = dim3(blocks);
+    cfg.blockDim = dim3(kThreads);
+    cfg.dynamicSmemBytes = kStageBytes;
+    cfg.stream = g->stream;
+    cfg.attrs = attrs;
+    cfg.numAttrs = na;
+    GC_CUDA_TRY(cudaLaunchKernelEx(&cfg, k_count_persistent<PROF>, a));
     *blocks_out = blocks;
     return GC_OK;
 }
@@ -689,10 +910,39 @@ int launch(gc_graph *g, CArgs &a, int *blocks_out) {
 }  // namespace
 
 // Scratch of COUNT mode (allocated on first use, kept with the handle).
+namespace {
+// big vertices (degree > kPackMax), at most cap of them recorded
+__global__ void k_find_big(const int64_t *__restrict__ ro, int64_t n, uint32_t *big, int cap,
+                           unsigned long long *nbig) {
+    for (int64_t v = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; v < n;
+         v += (int64_t)gridDim.x * blockDim.x) {
+        if (ro[v + 1] - ro[v] > kPackMax) {
+            const unsigned long long i = atomicAdd(nbig, 1ull);
+            if (i < (unsigned long long)cap) big[i] = (uint32_t)v;
+        }
+    }
+}
+}  // namespace
+
 int ensure_count_scratch(gc_graph *g) {
     Scratch &s = g->s;
     const size_t nn = (size_t)std::max<int64_t>(g->n, 1);
     if (s.cnt) return GC_OK;
+    // big vertices: seed-independent, found once per graph
+    GC_CUDA_TRY(dmalloc(&s.big, (size_t)(kHTab / 2) * 4));
+    GC_CUDA_TRY(dmalloc(&s.big32, (size_t)(3 * kHTab) * 4));
+    GC_CUDA_TRY(dmalloc(&s.cnt32, nn * 4));
+    {
+        unsigned long long *d = nullptr, h = 0;
+        GC_CUDA_TRY(dmalloc(&d, 8));
+        GC_CUDA_TRY(cudaMemsetAsync(d, 0, 8, g->stream));
+        if (g->n > 0)
+            k_find_big<<<g->sm_count * 4, 256, 0, g->stream>>>(g->ro, g->n, s.big, kHTab / 2, d);
+        GC_CUDA_TRY(cudaMemcpyAsync(&h, d, 8, cudaMemcpyDeviceToHost, g->stream));
+        GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
+        dfree(d);
+        s.nbig = h <= (unsigned long long)(kHTab / 2) ? (int)h : -1;  // -1: too many (EVENT mode)
+    }
     GC_CUDA_TRY(dmalloc(&s.cnt, nn * 8));
     GC_CUDA_TRY(dmalloc(&s.Z, nn * 4));
     s.sl_cap = (int64_t)nn;
@@ -712,6 +962,10 @@ int run_count_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     if (n == 0) return GC_OK;
     int rc = ensure_count_scratch(g);
     if (rc) return rc;
+    if (s.nbig < 0) {  // more big vertices than the shared hash set holds: witness kernel
+        rc = ensure_scratch(g, true, false);
+        return rc ? rc : run_persistent_maxmin(g, p, r);
+    }
     const int64_t max_rounds = std::min<int64_t>(std::min<int64_t>(p.max_rounds, 0xFFFFFFF0ll),
                                                  n / 2 + 2);
     rc = ensure_nk(g, std::min<int64_t>(std::min<int64_t>(n + 2, max_rounds + 2), 1 << 20));
@@ -742,6 +996,10 @@ int run_count_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     a.ci = g->ci;
     a.C = s.C;
     a.cnt = s.cnt;
+    a.cnt32 = s.cnt32;
+    a.big32 = s.big32;
+    a.big = s.big;
+    a.nbig = std::max(s.nbig, 0);
     a.Zlo = s.Z;
     a.SL = reinterpret_cast<Item *>(s.SL);
     a.WL = reinterpret_cast<Item *>(s.WL);

@@ -63,6 +63,10 @@ struct Scratch {
     int64_t *host_pinned = nullptr;  // pinned readback area
     // COUNT mode (gc_count.cu)
     unsigned long long *cnt = nullptr;   // (hi << 32) | lo uncoloured-neighbour counts
+    uint32_t *cnt32 = nullptr;           // packed (hi << 16) | lo counts (degree <= 65535)
+    uint32_t *big = nullptr;             // vertices of degree > 65535
+    uint32_t *big32 = nullptr;           // their per-side counts and flags
+    int nbig = 0;                        // their number (-1: too many to pack)
     uint32_t *Z = nullptr;               // Zlo: round from which lo is free (freed second)
     void *SL = nullptr;                  // short-row items (16 B)
     void *WL = nullptr;                  // long-row segment items (16 B)

@@ -51,6 +51,20 @@ __global__ void __launch_bounds__(512, 1) k_burst(unsigned long long *c64, uint3
                 for (int q = 0; q < 8; ++q) o[q] = __ldcg(c64 + w[q]);
 #pragma unroll
                 for (int q = 0; q < 8; ++q) acc += o[q];
+            } else if (MODE == 4) {  // 32-bit atom.add on a 2x larger footprint (stride 2)
+                uint32_t o[8];
+#pragma unroll
+                for (int q = 0; q < 8; ++q)
+                    asm volatile("atom.global.add.u32 %0, [%1], %2;" : "=r"(o[q]) : "l"(reinterpret_cast<uint32_t *>(c64) + 2 * (size_t)w[q]), "r"(~0u));
+#pragma unroll
+                for (int q = 0; q < 8; ++q) acc += o[q];
+            } else if (MODE == 5) {  // 64-bit atom.add on half the footprint
+                unsigned long long o[8];
+#pragma unroll
+                for (int q = 0; q < 8; ++q)
+                    asm volatile("atom.global.add.u64 %0, [%1], %2;" : "=l"(o[q]) : "l"(c64 + (w[q] >> 1)), "l"(~0ull));
+#pragma unroll
+                for (int q = 0; q < 8; ++q) acc += o[q];
             } else {  // contiguous 32-bit loads (a row segment): 8 x 128 B per warp
                 const uint32_t *row = c32 + ((size_t)w[0] & ~1023ull);
                 uint32_t o[8];
@@ -94,15 +108,17 @@ int main() {
     cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, 0);
     int clk = 0;
     cudaDeviceGetAttribute(&clk, cudaDevAttrClockRate, 0);
-    const char *names[4] = {"atom.add.u64 (ret)", "atom.add.u32 (ret)", "ld.u64 random", "ld.u32 contiguous rows"};
-    for (int mode = 0; mode < 4; ++mode) {
+    const char *names[6] = {"atom.add.u64 (ret) 134MB", "atom.add.u32 (ret) 67MB", "ld.u64 random 134MB",
+                            "ld.u32 contiguous rows", "atom.add.u32 (ret) 134MB", "atom.add.u64 (ret) 67MB"};
+    for (int mode = 0; mode < 6; ++mode) {
         for (int aw : {100, 800, 2368}) {
             cudaMemset(sum, 0, 8);
             cudaMemset(mx, 0, reps * 8);
             int active = aw;
             void *args[] = {&c64, &c32, &idx, (void *)&reps, &active, &sum, &mx};
             void *fn = mode == 0 ? (void *)k_burst<0> : mode == 1 ? (void *)k_burst<1>
-                     : mode == 2 ? (void *)k_burst<2> : (void *)k_burst<3>;
+                     : mode == 2 ? (void *)k_burst<2> : mode == 3 ? (void *)k_burst<3>
+                     : mode == 4 ? (void *)k_burst<4> : (void *)k_burst<5>;
             cudaLaunchCooperativeKernel(fn, sms, 512, args, 0, 0);
             cudaError_t e = cudaDeviceSynchronize();
             unsigned long long hs = 0;
@@ -113,7 +129,7 @@ int main() {
             for (int r = 10; r < reps; ++r) mmax += hm[r];
             mmax /= (reps - 10);
             const double cyc_ns = 1e6 / clk;  // clk in kHz
-            printf("%-24s warps %5d (x8 per lane = %7d accesses): mean warp %.0f ns, max warp %.0f ns  %s\n",
+            printf("%-28s warps %5d (x8 per lane = %7d accesses): mean warp %.0f ns, max warp %.0f ns  %s\n",
                    names[mode], aw, aw * 256, (double)hs / ((double)reps * aw) * cyc_ns, mmax * cyc_ns,
                    e == cudaSuccess ? "" : cudaGetErrorString(e));
         }
