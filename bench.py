@@ -126,14 +126,16 @@ def measured_peaks():
         return 6650.0, "fallback (B200_PROFILING.md 6.65 TB/s)"
 
 
-def ncu_traffic(workload: str):
+def ncu_traffic(workload: str, kernel: str):
     """Per-launch DRAM bytes of the dominant kernel from a committed ncu
-    --set full capture (profiles/ncu_traffic.json), or None."""
+    --set full capture (profiles/ncu_traffic.json) of that same kernel, or None."""
     try:
         with open(os.path.join(ROOT, "profiles", "ncu_traffic.json")) as f:
             d = json.load(f)
         ent = d.get(workload)
-        return None if ent is None else ent.get("dram_bytes_per_launch")
+        if ent is None or ent.get("kernel") != kernel:
+            return None
+        return ent.get("dram_bytes_per_launch")
     except Exception:
         return None
 
@@ -293,7 +295,7 @@ def main():
         kms, kl, kb = sp.kernel_ms[cls], sp.kernel_launches[cls], sp.kernel_bytes[cls]
         achieved = (kb / 1e9) / (kms / 1e3) if kms > 0 else 0.0
         roof = {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
-                "frac": achieved / peak, "traffic": ncu_traffic(f"rmat-s{scale}-{args.variant}"),
+                "frac": achieved / peak, "traffic": ncu_traffic(f"rmat-s{scale}-{args.variant}", name),
                 "kernel": name, "launches": kl, "avg_launch_us": 1e3 * kms / max(kl, 1),
                 "bytes_per_launch": kb / max(kl, 1), "kernel_share_of_step":
                 kms / max(sp.ms, 1e-9), "peak_source": peak_src,

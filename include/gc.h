@@ -87,8 +87,8 @@ typedef enum gc_status {
                                       little overhead, so keep it out of timed runs) */
 
 /* Sweep strategy (gc_options.mode).  All modes return identical colours. */
-#define GC_MODE_AUTO 0   /* max-min: SWEEP if max degree <= 32, else COUNT;
-                            multi-hash and Luby: SWEEP */
+#define GC_MODE_AUTO 0   /* max-min and multi-hash: SWEEP if max degree <= 8
+                            (meshes), else COUNT; Luby-MIS: COUNT */
 #define GC_MODE_SWEEP 1  /* every round re-scans each uncoloured vertex's row
                             with early exit (the paper's ComputeOp shape) */
 #define GC_MODE_EVENT 2  /* work-efficient: per-vertex witnesses + resume
@@ -100,7 +100,16 @@ typedef enum gc_status {
                             larger / smaller neighbours; each row is walked
                             once, when its vertex is coloured (one atomic per
                             entry); one persistent kernel, one grid barrier
-                            per round */
+                            per round.  Luby-MIS: the same
+                            colouring (first-fit greedy in decreasing weight
+                            order, R10) as a Jones-Plassmann wavefront over
+                            predecessor counts; a vertex's colour is the mex
+                            of its predecessors' colours;
+                            gc_stats.rounds / inner_iterations are then the
+                            wavefront depth, not Alg.3's iteration count.
+                            Multi-hash: H count pairs per vertex, the
+                            decision of a vertex kept as its first free
+                            (round, j, side) */
 
 typedef struct gc_graph gc_graph;
 

@@ -351,6 +351,7 @@ static void free_scratch(Scratch &s) {
     dfree(s.WL);
     dfree(s.hubs);
     dfree(s.cctr);
+    dfree(s.jslot);
     if (s.host_pinned) hfree(s.host_pinned);
     s = Scratch();
 }
@@ -536,11 +537,17 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     // and the plain sweep is fastest (measured: 128^3 mesh 0.47 ms sweep vs
     // 0.77 ms event); skewed graphs take thousands of rounds and need the
     // work-efficient event mode (R-MAT s24: 107 ms event vs 1689 ms sweep).
-    if (mode == GC_MODE_AUTO) mode = g->max_deg <= 32 ? GC_MODE_SWEEP : GC_MODE_COUNT;
-    if (luby) mode = GC_MODE_SWEEP;
-    if (mode != GC_MODE_SWEEP && H != 1) mode = GC_MODE_SWEEP;
+    // Luby-MIS: SWEEP runs Alg.2 + Alg.3 literally; COUNT computes the same
+    // colouring (first-fit greedy in decreasing weight order, R10) as a
+    // Jones-Plassmann wavefront over predecessor counts -- AUTO takes it.
+    // Measured (profiles/r01_configs.jsonl): COUNT wins on ER (0.79 vs 1.83 ms),
+    // rgg (0.66 vs 1.31) and R-MAT (35.6 vs 1689); the plain sweep only on
+    // meshes (128^3: 0.47 vs 0.57), whose rounds are few and uniform.
+    if (mode == GC_MODE_AUTO) mode = (luby || g->max_deg > 8) ? GC_MODE_COUNT : GC_MODE_SWEEP;
+    if (luby && mode != GC_MODE_COUNT) mode = GC_MODE_SWEEP;
+    if (H != 1 && mode != GC_MODE_COUNT) mode = GC_MODE_SWEEP;  // multi-hash: SWEEP or COUNT
 
-    int rc = ensure_scratch(g, mode == GC_MODE_EVENT || mode == GC_MODE_EVENT_MULTI, luby);
+    int rc = ensure_scratch(g, mode == GC_MODE_EVENT || mode == GC_MODE_EVENT_MULTI, luby);  // luby: S is also the fallback's
     if (rc) return rc;
     RunParams p;
     p.H = H;
@@ -559,7 +566,9 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     GC_CUDA_TRY(cudaEventCreate(&e1));
     GC_CUDA_TRY(cudaEventRecord(e0, g->stream));
     RunResult res;
-    if (luby)
+    if (luby && mode == GC_MODE_COUNT)
+        rc = g->count_unsafe ? GC_ERR_NOT_SYMMETRIC : run_count_jp(g, p, &res);
+    else if (luby)
         rc = run_luby(g, p, &res);
     else if (mode == GC_MODE_EVENT)
         rc = run_persistent_maxmin(g, p, &res);
@@ -575,9 +584,17 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
         // underflow or a stall -- never as a silently wrong colour, DESIGN.md
         // 7.0).  The witness kernel only needs the adjacency set: rerun there.
         g->count_unsafe = true;
-        mode = GC_MODE_EVENT;
-        rc = ensure_scratch(g, true, false);
-        if (!rc) rc = run_persistent_maxmin(g, p, &res);
+        if (luby) {
+            mode = GC_MODE_SWEEP;
+            rc = run_luby(g, p, &res);
+        } else if (H != 1) {
+            mode = GC_MODE_SWEEP;
+            rc = run_sweep_maxmin(g, p, &res);
+        } else {
+            mode = GC_MODE_EVENT;
+            rc = ensure_scratch(g, true, false);
+            if (!rc) rc = run_persistent_maxmin(g, p, &res);
+        }
     }
     if (rc) {
         cudaEventDestroy(e0);

@@ -100,6 +100,7 @@ enum : int {
     cVis = 210,     // PROF: entries walked in the rounds
     cPhaseNs = 211, // PROF: ns in the init phase, the rounds
     cHubs = 224,    // k_count: hub rows
+    cSlot = 240,    // JP: mex slots handed out (monotone)
     kCCtrWords = 256
 };
 
@@ -124,7 +125,16 @@ struct CArgs {
     uint32_t key;
     uint32_t max_rounds;
     unsigned long long sl_cap, wl_cap;
+    uint32_t *jslot;               // JP: mex slots of long rows (kSlotWords each)
+    unsigned long long jslot_cap;
+    int H;                         // MH: weight functions (count words v * H + j)
+    uint32_t mkeys[GC_MAX_HASHES]; // MH: their keys K_j
 };
+// JP mex slot of a long row: a 1024-bit presence set of its predecessors'
+// colours + the number of its entries not yet walked (the segment that takes
+// it to zero computes the mex and writes the colour).
+constexpr int kSlotWords = 36;  // [0, 32) bits, [32] entries remaining
+constexpr uint32_t kMexWin = 1024;
 
 __device__ __forceinline__ void flag_error(const CArgs &a, unsigned kind, uint32_t k, uint32_t v) {
     if (atomicCAS(&a.ctr[cErr], 0ull, (unsigned long long)kind) == 0ull) {
@@ -219,6 +229,7 @@ struct Stage {
     Item w[kStW];
     uint2 fresh[kStF];              // (w, lo side?) this block scheduled in the round
     uint32_t htab[kHTab];           // hash set of the big vertices (kNone = empty)
+    uint32_t wbits[kThreads / 32][32];  // JP: per-warp 1024-bit mex window
     struct Long {                   // schedule_fresh: a long row to expand
         int64_t rs, dst;            // row start; first item slot (>= 0 staged, < 0: ~global)
         uint32_t w, len, flags, pad;
@@ -322,9 +333,26 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
         red_max(prs + 8, gtimer() - t_round);
 }
 
+// JP: a mex slot for the long row of w (deg entries): cleared, its
+// remaining-entry count set, its index kept in Zlo[w] (JP has no lo side).
+__device__ __forceinline__ void jp_slot_init(const CArgs &a, uint32_t w, int64_t deg) {
+    const unsigned long long s = atom_add_global(a.ctr + cSlot, 1ull);
+    if (s >= a.jslot_cap) {
+        flag_error(a, 6, 0, w);
+        return;
+    }
+    uint4 *p = reinterpret_cast<uint4 *>(a.jslot + s * kSlotWords);
+#pragma unroll
+    for (int i = 0; i < kSlotWords / 4; ++i) p[i] = make_uint4(0u, 0u, 0u, 0u);
+    a.jslot[s * kSlotWords + 32] = (uint32_t)deg;
+    a.Zlo[w] = (uint32_t)s;
+}
+
 // Whole warp converged: schedule the rows of the lanes with `pred` (vertex w,
 // row [rs, rs + len)) for the next round: short rows as one SL item, longer
-// rows as ceil(len / kSeg) WL items (expanded by the whole warp).
+// rows as ceil(len / kSeg) WL items (expanded by the whole warp).  JP: every
+// segment of a row to be coloured carries the flags (each feeds the mex).
+template <bool JP>
 __device__ __forceinline__ void schedule_rows(const CArgs &a, bool pred, uint32_t w, int64_t rs,
                                               int64_t len, uint32_t ff) {
     const bool shortrow = pred && len <= kShortMax;
@@ -345,6 +373,7 @@ __device__ __forceinline__ void schedule_rows(const CArgs &a, bool pred, uint32_
         const int64_t r0 = __shfl_sync(kFull, rs, src);
         const int64_t ln = __shfl_sync(kFull, len, src);
         const uint32_t fs = __shfl_sync(kFull, ff, src);
+        if (JP && (fs & kFirst) && lane_id() == 0) jp_slot_init(a, ww, ln);
         const uint32_t nseg = (uint32_t)((ln + kSeg - 1) / kSeg);
         for (uint32_t q0 = 0; q0 < nseg; q0 += 32) {
             const uint32_t q = q0 + lane_id();
@@ -352,7 +381,7 @@ __device__ __forceinline__ void schedule_rows(const CArgs &a, bool pred, uint32_
             si.v = ww;
             const int64_t e0 = r0 + (int64_t)q * kSeg;
             si.e0 = e0;
-            si.lf = (uint32_t)min((int64_t)kSeg, r0 + ln - e0) | (q == 0 ? fs : 0u);
+            si.lf = (uint32_t)min((int64_t)kSeg, r0 + ln - e0) | ((q == 0 || JP) ? fs : 0u);
             stage_append(a, q < nseg, si, 1);
         }
     }
@@ -360,9 +389,10 @@ __device__ __forceinline__ void schedule_rows(const CArgs &a, bool pred, uint32_
 
 // Out-of-line copy for the rare paths inside the unrolled walk (overflowing
 // fresh list): keeps walk's code and registers small.
+template <bool JP>
 __device__ __noinline__ void schedule_rows_slow(const CArgs &a, bool pred, uint32_t w, int64_t rs,
                                                 int64_t len, uint32_t ff) {
-    schedule_rows(a, pred, w, rs, len, ff);
+    schedule_rows<JP>(a, pred, w, rs, len, ff);
 }
 
 // Colour v in round k (its scheduled round): min (2k+1) if the lo side is
@@ -376,16 +406,23 @@ __device__ __forceinline__ void colour(const CArgs &a, uint32_t v, uint32_t lf, 
 // in round k (v == kNone: idle lane; whole warp converged): decrement the
 // side of each neighbour w that v belongs to; a side reaching zero is free
 // from round k+1 and schedules w (first time only).
-template <int Q>
+// JP (the Luby-MIS variant as first-fit greedy in decreasing weight order,
+// R10): only the hi side exists (lo is pinned at 1); the entries w LARGER than
+// v are v's already-coloured predecessors -- their colours go into v's mex
+// set: bits < 64 of `mask` (short rows), or bits < 1024 of the warp's shared
+// bitmap `sbits` (WIDE: long-row segments).  mex = `want_mex` lanes only.
+template <int Q, bool JP = false, bool WIDE = false>
 __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, int64_t e,
-                                     int64_t end, int stride, uint32_t k, uint32_t &nvis) {
+                                     int64_t end, int stride, uint32_t k, uint32_t &nvis,
+                                     unsigned long long *mask = nullptr, uint32_t *sbits = nullptr,
+                                     bool want_mex = false) {
     uint32_t w[Q];
 #pragma unroll
     for (int q = 0; q < Q; ++q) {
         const int64_t eq = e + (int64_t)q * stride;
         w[q] = (v != kNone && eq < end) ? __ldcs(a.ci + eq) : kNone;
     }
-    // One 32-bit atomic per entry, address and value chosen without a branch
+    // One atomic per entry, address and value chosen without a branch
     // (a branch around each atomic made the compiler wait for every result).
 #if GC_PACKED
     uint32_t old[Q];
@@ -394,11 +431,13 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
 #endif
     bool hi[Q];
     int slot[Q];
+    uint32_t cv[Q];  // JP: colours of the larger neighbours
 #pragma unroll
     for (int q = 0; q < Q; ++q) {
         const bool live = w[q] != kNone;
         const uint32_t wq = live ? w[q] : 0u;
         hi[q] = live && pv > weight_mix(wq ^ a.key);  // v is a larger neighbour of w
+        cv[q] = kNone;
 #if GC_PACKED
         slot[q] = (live && a.nbig > 0) ? big_slot(wq) : -1;
         uint32_t *adr = slot[q] >= 0 ? a.big32 + 2 * slot[q] + (hi[q] ? 0 : 1) : a.cnt32 + wq;
@@ -406,8 +445,27 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
         old[q] = live ? atom_add_global32(adr, dec) : 2u;
 #else
         slot[q] = -1;
-        old[q] = live ? atom_add_global(a.cnt + wq, hi[q] ? kDecHi : kDecLo) : 2ull;
+        if (JP) {
+            old[q] = hi[q] ? atom_add_global(a.cnt + wq, kDecHi) : 2ull;
+            if (live && !hi[q] && want_mex) cv[q] = __ldcg(a.C + wq);
+        } else {
+            old[q] = live ? atom_add_global(a.cnt + wq, hi[q] ? kDecHi : kDecLo) : 2ull;
+        }
 #endif
+    }
+    if (JP && want_mex) {
+#pragma unroll
+        for (int q = 0; q < Q; ++q) {
+            const uint32_t c = cv[q];
+            if (w[q] != kNone && !hi[q]) {
+                if (c == GC_UNC) flag_error(a, 5, k, v);  // a predecessor is uncoloured
+                if (WIDE) {
+                    if (c < 1024u) atomicOr(sbits + (c >> 5), 1u << (c & 31u));
+                } else if (c < 64u) {
+                    *mask |= 1ull << c;
+                }
+            }
+        }
     }
     bool fresh[Q];
 #pragma unroll
@@ -459,9 +517,91 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
                 rs = a.ro[w[q]];
                 re = a.ro[w[q] + 1];
             }
-            schedule_rows_slow(a, ovf[q], w[q], rs, re - rs, kFirst | (hi[q] ? 0u : kLoSide));
+            schedule_rows_slow<JP>(a, ovf[q], w[q], rs, re - rs, kFirst | (hi[q] ? 0u : kLoSide));
         }
     }
+}
+
+// MH (multi-hash, H weight functions, R8): walk the row of v coloured in
+// round k; per entry w and per j decrement hi_j(w) or lo_j(w).  A side (j, s)
+// reaching zero is free from round k+1: it records the code
+// (k+1) << 5 | j << 1 | (s == hi) with atomicMin in Zlo[w], so Zlo[w] ends up
+// holding w's decision -- its first free round, the smallest j free then, the
+// min colour if that j's lo side is free (R8, R9) -- and sides freed in
+// later rounds never override it.  The atomicMin that replaces kNever
+// schedules w (exactly one per vertex).
+template <int Q>
+__device__ __forceinline__ void walk_mh(const CArgs &a, uint32_t v, int64_t e, int64_t end, int stride,
+                                        uint32_t k, uint32_t &nvis) {
+    uint32_t w[Q];
+#pragma unroll
+    for (int q = 0; q < Q; ++q) {
+        const int64_t eq = e + (int64_t)q * stride;
+        w[q] = (v != kNone && eq < end) ? __ldcs(a.ci + eq) : kNone;
+    }
+    const int H = a.H;
+    uint32_t pv[GC_MAX_HASHES];
+#pragma unroll
+    for (int j = 0; j < GC_MAX_HASHES; ++j) pv[j] = j < H ? weight_mix(v ^ a.mkeys[j]) : 0u;
+    bool fresh[Q];
+#pragma unroll
+    for (int q = 0; q < Q; ++q) {
+        fresh[q] = false;
+        if (w[q] == kNone) continue;
+        ++nvis;
+        unsigned long long *cw = a.cnt + (size_t)w[q] * H;
+        unsigned long long old[GC_MAX_HASHES];
+        bool hi[GC_MAX_HASHES];
+#pragma unroll
+        for (int j = 0; j < GC_MAX_HASHES; ++j) {
+            if (j < H) {
+                hi[j] = pv[j] > weight_mix(w[q] ^ a.mkeys[j]);
+                old[j] = atom_add_global(cw + j, hi[j] ? kDecHi : kDecLo);
+            }
+        }
+#pragma unroll
+        for (int j = 0; j < GC_MAX_HASHES; ++j) {
+            if (j < H) {
+                const uint32_t side = hi[j] ? (uint32_t)(old[j] >> 32) : (uint32_t)old[j];
+                if (side == 1u) {
+                    const uint32_t code = ((k + 1u) << 5) | ((uint32_t)j << 1) | (hi[j] ? 1u : 0u);
+                    if (atomicMin(a.Zlo + w[q], code) == kNever) fresh[q] = true;
+                } else if (side == 0u) {
+                    flag_error(a, 4, k, w[q]);
+                }
+            }
+        }
+    }
+    bool ovf[Q];
+#pragma unroll
+    for (int q = 0; q < Q; ++q) {
+        ovf[q] = false;
+        if (fresh[q]) {
+            asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ro + w[q]));
+            const unsigned pos = atomicAdd(&stage().nf, 1u);
+            if (pos < (unsigned)kStF) stage().fresh[pos] = make_uint2(w[q], 0u);
+            else ovf[q] = true;
+        }
+    }
+#pragma unroll
+    for (int q = 0; q < Q; ++q) {
+        if (__any_sync(kFull, ovf[q])) {
+            int64_t rs = 0, re = 0;
+            if (ovf[q]) {
+                rs = a.ro[w[q]];
+                re = a.ro[w[q] + 1];
+            }
+            schedule_rows_slow<false>(a, ovf[q], w[q], rs, re - rs, kFirst);
+        }
+    }
+}
+
+// MH: colour v in its scheduled round k from the decision code in Zlo[v]
+__device__ __forceinline__ void colour_mh(const CArgs &a, uint32_t v, uint32_t k) {
+    const uint32_t code = __ldcg(a.Zlo + v);
+    if ((code >> 5) != k) flag_error(a, 8, k, v);
+    const uint32_t j = (code >> 1) & 15u;
+    a.C[v] = 2u * (k * (uint32_t)a.H + j) + ((code & 1u) ? 0u : 1u);
 }
 
 // Whole block, end of a round: stage the items of the vertices on the fresh
@@ -469,6 +609,7 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
 // then the segments of all long rows written by the whole block.  An SL
 // overflow, a long row that does not fit the staged WL buffer and a long-row
 // list overflow go straight to the global lists (rare).
+template <bool JP>
 __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nullptr,
                                                unsigned long long t_round = 0) {
     Stage &st = stage();
@@ -505,6 +646,7 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
                 else flag_error(a, 1, 0, f.x);
             }
         } else {
+            if (JP) jp_slot_init(a, f.x, len);
             const uint32_t nseg = (uint32_t)((len + kSeg - 1) / kSeg);
             const unsigned sb = atomicAdd(&st.n[1], nseg);
             int64_t dst;
@@ -527,7 +669,7 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
                     Item si;
                     si.v = f.x;
                     si.e0 = rs + (int64_t)q * kSeg;
-                    si.lf = (uint32_t)min((int64_t)kSeg, len - (int64_t)q * kSeg) | (q == 0 ? fl : 0u);
+                    si.lf = (uint32_t)min((int64_t)kSeg, len - (int64_t)q * kSeg) | ((q == 0 || JP) ? fl : 0u);
                     if (dst >= 0) st.w[dst + q] = si;
                     else a.WL[~dst + q] = si;
                 }
@@ -543,7 +685,7 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
             Item si;
             si.v = L.w;
             si.e0 = L.rs + (int64_t)q * kSeg;
-            si.lf = (uint32_t)min((int64_t)kSeg, (int64_t)L.len - (int64_t)q * kSeg) | (q == 0 ? L.flags : 0u);
+            si.lf = (uint32_t)min((int64_t)kSeg, (int64_t)L.len - (int64_t)q * kSeg) | ((q == 0 || JP) ? L.flags : 0u);
             if (L.dst >= 0) st.w[L.dst + q] = si;
             else a.WL[~L.dst + q] = si;
         }
@@ -565,7 +707,83 @@ __device__ __forceinline__ void set_targets(const CArgs &a, uint32_t k, unsigned
     __syncthreads();
 }
 
-template <bool PROF>
+// JP, whole warp converged: this long-row segment of v has put its
+// predecessors' colours into the warp's window `sb`; merge it into v's slot
+// and retire its entries; the segment that retires the last entry computes
+// the mex and colours v (first-fit, R10).
+__device__ __noinline__ uint32_t jp_mex_rescan(const CArgs &a, uint32_t v, uint32_t pv, uint32_t *sb);
+
+__device__ __forceinline__ void jp_segment_done(const CArgs &a, uint32_t v, uint32_t len, uint32_t pv,
+                                                uint32_t *sb, uint32_t k) {
+    const unsigned lane = lane_id();
+    __syncwarp();
+    const uint32_t slot = __ldcg(a.Zlo + v);
+    uint32_t *S = a.jslot + (size_t)slot * kSlotWords;
+    const uint32_t word = sb[lane];
+    if (word) atomicOr(S + lane, word);
+    __threadfence();
+    __syncwarp();
+    uint32_t last = 0;
+    if (lane == 0) {
+        uint32_t old;
+        asm volatile("atom.acq_rel.gpu.global.add.u32 %0, [%1], %2;"
+                     : "=r"(old) : "l"(S + 32), "r"(0u - len) : "memory");
+        last = old == len ? 1u : 0u;
+        if (old < len) flag_error(a, 7, k, v);
+    }
+    last = __shfl_sync(kFull, last, 0);
+    if (!last) return;
+    __threadfence();
+    const uint32_t bw = __ldcg(S + lane);
+    const unsigned nf = __ballot_sync(kFull, bw != 0xFFFFFFFFu);
+    uint32_t mex;
+    if (nf) {
+        const int f = __ffs(nf) - 1;
+        mex = 32u * (uint32_t)f + (uint32_t)(__ffs(~__shfl_sync(kFull, bw, f)) - 1);
+    } else {
+        mex = jp_mex_rescan(a, v, pv, sb);
+    }
+    if (lane == 0) {
+        a.C[v] = mex;
+        atomicAdd(&stage().colored, 1u);
+    }
+}
+
+// mex >= kMexWin (a vertex with >= 1024 predecessors of distinct colours):
+// the warp rescans the row for successive 1024-colour windows (rare).
+__device__ __noinline__ uint32_t jp_mex_rescan(const CArgs &a, uint32_t v, uint32_t pv, uint32_t *sb) {
+    const unsigned lane = lane_id();
+    const int64_t rs = a.ro[v], re = a.ro[v + 1];
+    for (uint32_t b = kMexWin;; b += kMexWin) {
+        __syncwarp();
+        sb[lane] = 0u;
+        __syncwarp();
+        for (int64_t e = rs + lane; e < re; e += 32) {
+            const uint32_t u = a.ci[e];
+            if (weight_mix(u ^ a.key) > pv) {
+                const uint32_t c = __ldcg(a.C + u) - b;
+                if (c < kMexWin) atomicOr(sb + (c >> 5), 1u << (c & 31u));
+            }
+        }
+        __syncwarp();
+        const uint32_t bw = sb[lane];
+        const unsigned nf = __ballot_sync(kFull, bw != 0xFFFFFFFFu);
+        if (nf) {
+            const int f = __ffs(nf) - 1;
+            return b + 32u * (uint32_t)f + (uint32_t)(__ffs(~__shfl_sync(kFull, bw, f)) - 1);
+        }
+    }
+}
+
+// 8-lane groups: OR of the group's masks
+__device__ __forceinline__ unsigned long long group8_or(unsigned long long m) {
+    m |= __shfl_xor_sync(kFull, m, 1);
+    m |= __shfl_xor_sync(kFull, m, 2);
+    m |= __shfl_xor_sync(kFull, m, 4);
+    return m;
+}
+
+template <bool PROF, bool JP, bool MH>
 __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
     const unsigned lane = lane_id();
     const unsigned long long gtid = (unsigned long long)blockIdx.x * blockDim.x + threadIdx.x;
@@ -606,13 +824,24 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
     for (unsigned long long base = gwarp * 32; base < (unsigned long long)n; base += nwarps * 32) {
         const uint32_t v = (uint32_t)(base + lane);
         const bool valid = (int64_t)(base + lane) < n;
-        const unsigned long long c = valid ? a.cnt[v] : 0x100000001ull;
-        const uint32_t hi = (uint32_t)(c >> 32), lo = (uint32_t)c;
-        const bool zero = valid && (hi == 0u || lo == 0u);
+        uint32_t hi = 1u, lo = 1u, code = kNever;
+        if (MH) {
+            // round 0: the smallest j with a free side, its min side first (R8, R9)
+            for (int j = 0; valid && j < a.H; ++j) {
+                const unsigned long long c = a.cnt[(size_t)v * a.H + j];
+                if ((uint32_t)c == 0u) code = min(code, (uint32_t)j << 1);
+                else if ((uint32_t)(c >> 32) == 0u) code = min(code, ((uint32_t)j << 1) | 1u);
+            }
+        } else {
+            const unsigned long long c = valid ? a.cnt[v] : 0x100000001ull;
+            hi = (uint32_t)(c >> 32);
+            lo = (uint32_t)c;
+        }
+        const bool zero = valid && (MH ? code != kNever : (hi == 0u || lo == 0u));
         int64_t rs = 0, re = 0;
         if (valid) {
             const int sl = (GC_PACKED && a.nbig > 0) ? big_slot(v) : -1;
-            if (!GC_PACKED) {
+            if (!GC_PACKED || MH) {
             } else if (sl < 0) {
                 a.cnt32[v] = (hi << 16) | lo;  // deg <= kPackMax
             } else {
@@ -620,8 +849,13 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
                 a.big32[2 * sl + 1] = lo;
                 a.big32[2 * kHTab + sl] = (hi == 0u || lo == 0u) ? 1u : 0u;
             }
-            a.Zlo[v] = kNever;
-            a.C[v] = zero ? (lo == 0u ? 1u : 0u) : GC_UNC;
+            if (MH) {
+                a.Zlo[v] = code;  // round 0's decision (not kNever: never rescheduled)
+                a.C[v] = zero ? 2u * (code >> 1) + ((code & 1u) ? 0u : 1u) : GC_UNC;
+            } else {
+                if (!JP) a.Zlo[v] = kNever;
+                a.C[v] = zero ? (lo == 0u ? 1u : 0u) : GC_UNC;
+            }
             if (zero) {
                 rs = a.ro[v];
                 re = a.ro[v + 1];
@@ -629,7 +863,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
         }
         const unsigned word = __ballot_sync(kFull, zero);
         if (lane == 0 && word) atomicAdd(&stage().colored, (unsigned)__popc(word));
-        schedule_rows(a, zero && re > rs, v, rs, re - rs, 0u);  // walked in round 0
+        schedule_rows<JP>(a, zero && re > rs, v, rs, re - rs, 0u);  // walked in round 0
     }
     stage_flush(a);
     if (!grid_barrier(a, 0)) return;
@@ -688,46 +922,81 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
                 Item it = a.WL[wl0 + u];
                 if (it.v == kNone) it.lf = 0;  // hole left by schedule_fresh
                 const uint32_t pv = weight_mix(it.v ^ a.key);
-                if ((it.lf & kFirst) && lane == 0) {
-                    colour(a, it.v, it.lf, k);
-                    atomicAdd(&stage().colored, 1u);
+                if (JP && (it.lf & kFirst)) {  // a segment of a row being coloured
+                    uint32_t *sb = stage().wbits[threadIdx.x >> 5];
+                    sb[lane] = 0u;
+                    __syncwarp();
+                    walk<kSeg / 32, true, true>(a, it.v, pv, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k,
+                                                nvis, nullptr, sb, true);
+                    jp_segment_done(a, it.v, it.lf & kLenMask, pv, sb, k);
+                } else {
+                    if (!JP && (it.lf & kFirst) && lane == 0) {
+                        if (MH) colour_mh(a, it.v, k);
+                        else colour(a, it.v, it.lf, k);
+                        atomicAdd(&stage().colored, 1u);
+                    }
+                    if (MH)
+                        walk_mh<kSeg / 32>(a, it.v, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k, nvis);
+                    else
+                        walk<kSeg / 32, JP>(a, it.v, pv, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k, nvis);
                 }
-                walk<kSeg / 32>(a, it.v, pv, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k, nvis);
             } else if (lane_rows) {
                 // short rows: one per lane, 4 entries per step
                 const unsigned long long idx = sl0 + 32 * (u - nw) + lane;
                 uint32_t v = kNone, len = 0, pv = 0;
                 int64_t e0 = 0;
+                bool want = false;
                 if (idx < sl1) {
                     const Item it = a.SL[idx];
                     v = it.v;
                     len = it.lf & kLenMask;
                     e0 = it.e0;
                     pv = weight_mix(v ^ a.key);
-                    if (it.lf & kFirst) {
-                        colour(a, v, it.lf, k);
+                    want = JP && (it.lf & kFirst);
+                    if (!JP && (it.lf & kFirst)) {
+                        if (MH) colour_mh(a, v, k);
+                        else colour(a, v, it.lf, k);
                         atomicAdd(&stage().colored, 1u);
                     }
                 }
-                for (uint32_t j = 0; __any_sync(kFull, j < len); j += 4)
-                    walk<4>(a, j < len ? v : kNone, pv, e0 + j, e0 + len, 1, k, nvis);
+                unsigned long long mask = 0ull;
+                for (uint32_t j = 0; __any_sync(kFull, j < len); j += 4) {
+                    if (MH) walk_mh<4>(a, j < len ? v : kNone, e0 + j, e0 + len, 1, k, nvis);
+                    else walk<4, JP>(a, j < len ? v : kNone, pv, e0 + j, e0 + len, 1, k, nvis, &mask, nullptr, want);
+                }
+                if (JP && want) {  // <= 32 predecessors: the mex is below 64
+                    a.C[v] = (uint32_t)(__ffsll((long long)~mask) - 1);
+                    atomicAdd(&stage().colored, 1u);
+                }
             } else {
                 // short rows: 4 per warp, 8 lanes each, 4 entries per lane
                 const unsigned long long idx = sl0 + 4 * (u - nw) + (lane >> 3);
                 uint32_t v = kNone, len = 0, pv = 0;
                 int64_t e0 = 0;
+                bool want = false;
                 if (idx < sl1) {
                     const Item it = a.SL[idx];
                     v = it.v;
                     len = it.lf & kLenMask;
                     e0 = it.e0;
                     pv = weight_mix(v ^ a.key);
-                    if ((it.lf & kFirst) && (lane & 7u) == 0u) {
-                        colour(a, v, it.lf, k);
+                    want = JP && (it.lf & kFirst);
+                    if (!JP && (it.lf & kFirst) && (lane & 7u) == 0u) {
+                        if (MH) colour_mh(a, v, k);
+                        else colour(a, v, it.lf, k);
                         atomicAdd(&stage().colored, 1u);
                     }
                 }
-                walk<4>(a, v, pv, e0 + (lane & 7u), e0 + len, 8, k, nvis);
+                unsigned long long mask = 0ull;
+                if (MH) walk_mh<4>(a, v, e0 + (lane & 7u), e0 + len, 8, k, nvis);
+                else walk<4, JP>(a, v, pv, e0 + (lane & 7u), e0 + len, 8, k, nvis, &mask, nullptr, want);
+                if (JP) {
+                    mask = group8_or(mask);
+                    if (want && (lane & 7u) == 0u) {
+                        a.C[v] = (uint32_t)(__ffsll((long long)~mask) - 1);
+                        atomicAdd(&stage().colored, 1u);
+                    }
+                }
             }
             if (prs && lane == 0)
                 red_max(prs + 10, (unsigned long long)(clock64() - c_unit));
@@ -740,7 +1009,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
             nvis_tot += nvis;
             nvis = 0;
         }
-        schedule_fresh(a, prs, t_round);
+        schedule_fresh<JP>(a, prs, t_round);
         stage_flush(a, prs, t_round);
         if (!grid_barrier(a, k)) return;
         if (PROF && gtid == 0) {
@@ -763,16 +1032,24 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
     }
 }
 
-// hi / lo counts of every vertex (round-0 state: everything is uncoloured).
+// hi / lo counts of every vertex (round-0 state: everything is uncoloured),
+// per weight function j < H (MH: the multi-hash variant; word v * H + j).
 // A warp takes 32 consecutive vertices: rows <= 16 one lane each, rows up to
 // kHubMin the whole warp (coalesced), longer rows go to the hub list.
+struct CountKeys {
+    uint32_t k[GC_MAX_HASHES];
+    int H;
+};
+
+template <bool MH>
 __global__ void __launch_bounds__(256) k_count(const int64_t *__restrict__ ro,
                                                const uint32_t *__restrict__ ci, int64_t n,
-                                               uint32_t key, unsigned long long *cnt,
-                                               uint2 *hubs, unsigned long long *nhubs) {
+                                               CountKeys keys, unsigned long long *cnt,
+                                               uint2 *hubs, unsigned long long *nhubs, int jp) {
     const unsigned lane = lane_id();
     const unsigned long long gw = ((unsigned long long)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const unsigned long long nw = ((unsigned long long)gridDim.x * blockDim.x) >> 5;
+    const int H = MH ? keys.H : 1;
     for (unsigned long long base = gw * 32; base < (unsigned long long)n; base += nw * 32) {
         const int64_t v = (int64_t)(base + lane);
         const bool valid = v < n;
@@ -782,19 +1059,22 @@ __global__ void __launch_bounds__(256) k_count(const int64_t *__restrict__ ro,
             re = ro[v + 1];
         }
         const int64_t deg = re - rs;
-        const uint32_t pv = weight_mix((uint32_t)v ^ key);
         if (valid && deg <= 16) {
-            uint32_t h = 0;
             uint32_t u[16];
 #pragma unroll
             for (int q = 0; q < 16; ++q) u[q] = q < deg ? __ldcs(ci + rs + q) : 0u;
+            for (int j = 0; j < H; ++j) {
+                const uint32_t key = keys.k[j];
+                const uint32_t pv = weight_mix((uint32_t)v ^ key);
+                uint32_t h = 0;
 #pragma unroll
-            for (int q = 0; q < 16; ++q) h += (q < deg && weight_mix(u[q] ^ key) > pv) ? 1u : 0u;
-            cnt[v] = ((unsigned long long)h << 32) | (unsigned long long)(deg - h);
+                for (int q = 0; q < 16; ++q) h += (q < deg && weight_mix(u[q] ^ key) > pv) ? 1u : 0u;
+                cnt[(size_t)v * H + j] = ((unsigned long long)h << 32) | (unsigned long long)(jp ? 1 : deg - h);
+            }
         }
         const bool big = valid && deg > kHubMin;
         if (big) {
-            cnt[v] = 0ull;  // k_count_hub adds the chunks
+            for (int j = 0; j < H; ++j) cnt[(size_t)v * H + j] = jp ? 1ull : 0ull;  // k_count_hub adds the chunks
             const int64_t nch = (deg + kHubChunk - 1) / kHubChunk;
             const unsigned long long b = atomicAdd(nhubs, (unsigned long long)nch);
             for (int64_t c = 0; c < nch; ++c)
@@ -805,60 +1085,70 @@ __global__ void __launch_bounds__(256) k_count(const int64_t *__restrict__ ro,
             const int src = __ffs(mid) - 1;
             mid &= mid - 1;
             const int64_t r0 = __shfl_sync(kFull, rs, src), r1 = __shfl_sync(kFull, re, src);
-            const uint32_t p = __shfl_sync(kFull, pv, src);
-            uint32_t h = 0;
-            for (int64_t e = r0 + lane; e < r1; e += 128) {
-                uint32_t u[4];
+            const uint32_t vs = (uint32_t)(base + src);
+            for (int j = 0; j < H; ++j) {
+                const uint32_t key = keys.k[j];
+                const uint32_t p = weight_mix(vs ^ key);
+                uint32_t h = 0;
+                for (int64_t e = r0 + lane; e < r1; e += 128) {
+                    uint32_t u[4];
 #pragma unroll
-                for (int q = 0; q < 4; ++q) u[q] = e + 32 * q < r1 ? __ldcs(ci + e + 32 * q) : 0u;
+                    for (int q = 0; q < 4; ++q) u[q] = e + 32 * q < r1 ? __ldcs(ci + e + 32 * q) : 0u;
 #pragma unroll
-                for (int q = 0; q < 4; ++q)
-                    h += (e + 32 * q < r1 && weight_mix(u[q] ^ key) > p) ? 1u : 0u;
+                    for (int q = 0; q < 4; ++q)
+                        h += (e + 32 * q < r1 && weight_mix(u[q] ^ key) > p) ? 1u : 0u;
+                }
+                h = __reduce_add_sync(kFull, h);
+                if (lane == (unsigned)src)
+                    cnt[(size_t)v * H + j] =
+                        ((unsigned long long)h << 32) | (unsigned long long)(jp ? 1 : deg - h);
             }
-            h = __reduce_add_sync(kFull, h);
-            if (lane == (unsigned)src)
-                cnt[v] = ((unsigned long long)h << 32) | (unsigned long long)(deg - h);
         }
     }
 }
 
 // Rows longer than kHubMin: one block per kHubChunk-entry chunk (the chunk
 // list (v, c) was written by k_count); partial counts are added atomically.
+template <bool MH>
 __global__ void __launch_bounds__(256) k_count_hub(const int64_t *__restrict__ ro,
-                                                   const uint32_t *__restrict__ ci, uint32_t key,
+                                                   const uint32_t *__restrict__ ci, CountKeys keys,
                                                    unsigned long long *cnt, const uint2 *hubs,
-                                                   const unsigned long long *nhubs) {
+                                                   const unsigned long long *nhubs, int jp) {
     __shared__ uint32_t red[8];
     const unsigned long long nh = *nhubs;
+    const int H = MH ? keys.H : 1;
     for (unsigned long long i = blockIdx.x; i < nh; i += gridDim.x) {
         const uint2 hc = hubs[i];
         const uint32_t v = hc.x;
         const int64_t rs = ro[v], re = ro[v + 1];
-        const uint32_t pv = weight_mix(v ^ key);
         const int64_t c0 = rs + (int64_t)hc.y * kHubChunk, c1 = min(re, c0 + (int64_t)kHubChunk);
-        uint32_t hcount = 0;
+        for (int j = 0; j < H; ++j) {
+            const uint32_t key = keys.k[j];
+            const uint32_t pv = weight_mix(v ^ key);
+            uint32_t hcount = 0;
 #pragma unroll 4
-        for (int64_t e = c0 + threadIdx.x; e < c1; e += blockDim.x)
-            hcount += weight_mix(__ldcs(ci + e) ^ key) > pv ? 1u : 0u;
-        hcount = __reduce_add_sync(kFull, hcount);
-        if (lane_id() == 0) red[threadIdx.x >> 5] = hcount;
-        __syncthreads();
-        if (threadIdx.x == 0) {
-            uint32_t t = 0;
-            for (int j = 0; j < (int)(blockDim.x >> 5); ++j) t += red[j];
-            const unsigned long long tot = (unsigned long long)(c1 - c0);
-            atomicAdd(&cnt[v], ((unsigned long long)t << 32) + (tot - t));
+            for (int64_t e = c0 + threadIdx.x; e < c1; e += blockDim.x)
+                hcount += weight_mix(__ldcs(ci + e) ^ key) > pv ? 1u : 0u;
+            hcount = __reduce_add_sync(kFull, hcount);
+            if (lane_id() == 0) red[threadIdx.x >> 5] = hcount;
+            __syncthreads();
+            if (threadIdx.x == 0) {
+                uint32_t t = 0;
+                for (int w = 0; w < (int)(blockDim.x >> 5); ++w) t += red[w];
+                const unsigned long long tot = (unsigned long long)(c1 - c0);
+                atomicAdd(&cnt[(size_t)v * H + j], ((unsigned long long)t << 32) + (jp ? 0ull : tot - t));
+            }
+            __syncthreads();
         }
-        __syncthreads();
     }
 }
 
-template <bool PROF>
+template <bool PROF, bool JP, bool MH>
 int launch(gc_graph *g, CArgs &a, int *blocks_out) {
     int per_sm = 0;
-    GC_CUDA_TRY(cudaFuncSetAttribute(k_count_persistent<PROF>,
+    GC_CUDA_TRY(cudaFuncSetAttribute(k_count_persistent<PROF, JP, MH>,
                                      cudaFuncAttributeMaxDynamicSharedMemorySize, (int)kStageBytes));
-    GC_CUDA_TRY(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_count_persistent<PROF>,
+    GC_CUDA_TRY(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_count_persistent<PROF, JP, MH>,
                                                               kThreads, kStageBytes));
     if (per_sm < 1) {
         set_error("persistent count kernel cannot be resident");
@@ -902,7 +1192,7 @@ int launch(gc_graph *g, CArgs &a, int *blocks_out) {
     cfg.stream = g->stream;
     cfg.attrs = attrs;
     cfg.numAttrs = na;
-    GC_CUDA_TRY(cudaLaunchKernelEx(&cfg, k_count_persistent<PROF>, a));
+    GC_CUDA_TRY(cudaLaunchKernelEx(&cfg, k_count_persistent<PROF, JP, MH>, a));
     *blocks_out = blocks;
     return GC_OK;
 }
@@ -911,16 +1201,30 @@ int launch(gc_graph *g, CArgs &a, int *blocks_out) {
 
 // Scratch of COUNT mode (allocated on first use, kept with the handle).
 namespace {
-// big vertices (degree > kPackMax), at most cap of them recorded
-__global__ void k_find_big(const int64_t *__restrict__ ro, int64_t n, uint32_t *big, int cap,
-                           unsigned long long *nbig) {
+// vertices of degree > dmin (big: > kPackMax; JP slots: > kShortMax),
+// counted, at most cap of them recorded
+__global__ void k_find_big(const int64_t *__restrict__ ro, int64_t n, int64_t dmin, uint32_t *big,
+                           int cap, unsigned long long *nbig) {
     for (int64_t v = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; v < n;
          v += (int64_t)gridDim.x * blockDim.x) {
-        if (ro[v + 1] - ro[v] > kPackMax) {
+        if (ro[v + 1] - ro[v] > dmin) {
             const unsigned long long i = atomicAdd(nbig, 1ull);
             if (i < (unsigned long long)cap) big[i] = (uint32_t)v;
         }
     }
+}
+
+// number of vertices of degree > dmin
+int count_deg_above(gc_graph *g, int64_t dmin, uint32_t *big, int cap, unsigned long long *out) {
+    unsigned long long *d = nullptr;
+    GC_CUDA_TRY(dmalloc(&d, 8));
+    GC_CUDA_TRY(cudaMemsetAsync(d, 0, 8, g->stream));
+    if (g->n > 0)
+        k_find_big<<<g->sm_count * 4, 256, 0, g->stream>>>(g->ro, g->n, dmin, big, cap, d);
+    GC_CUDA_TRY(cudaMemcpyAsync(out, d, 8, cudaMemcpyDeviceToHost, g->stream));
+    GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
+    dfree(d);
+    return GC_OK;
 }
 }  // namespace
 
@@ -933,15 +1237,10 @@ int ensure_count_scratch(gc_graph *g) {
     GC_CUDA_TRY(dmalloc(&s.big32, (size_t)(3 * kHTab) * 4));
     GC_CUDA_TRY(dmalloc(&s.cnt32, nn * 4));
     {
-        unsigned long long *d = nullptr, h = 0;
-        GC_CUDA_TRY(dmalloc(&d, 8));
-        GC_CUDA_TRY(cudaMemsetAsync(d, 0, 8, g->stream));
-        if (g->n > 0)
-            k_find_big<<<g->sm_count * 4, 256, 0, g->stream>>>(g->ro, g->n, s.big, kHTab / 2, d);
-        GC_CUDA_TRY(cudaMemcpyAsync(&h, d, 8, cudaMemcpyDeviceToHost, g->stream));
-        GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
-        dfree(d);
-        s.nbig = h <= (unsigned long long)(kHTab / 2) ? (int)h : -1;  // -1: too many (EVENT mode)
+        unsigned long long h = 0;
+        int rc = count_deg_above(g, kPackMax, s.big, kHTab / 2, &h);
+        if (rc) return rc;
+        s.nbig = h <= (unsigned long long)(kHTab / 2) ? (int)h : -1;  // -1: too many to pack
     }
     GC_CUDA_TRY(dmalloc(&s.cnt, nn * 8));
     GC_CUDA_TRY(dmalloc(&s.Z, nn * 4));
@@ -955,19 +1254,44 @@ int ensure_count_scratch(gc_graph *g) {
     return GC_OK;
 }
 
-int run_count_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
+// JP mex slots: one per vertex of degree > kShortMax (each is scheduled once)
+static int ensure_jp_scratch(gc_graph *g) {
+    Scratch &s = g->s;
+    if (s.jslot) return GC_OK;
+    unsigned long long h = 0;
+    int rc = count_deg_above(g, kShortMax, nullptr, 0, &h);
+    if (rc) return rc;
+    s.jslot_cap = (int64_t)h;
+    GC_CUDA_TRY(dmalloc(&s.jslot, ((size_t)h + 1) * kSlotWords * 4));
+    return GC_OK;
+}
+
+static int run_count(gc_graph *g, const RunParams &p, RunResult *r, bool jp) {
     Scratch &s = g->s;
     const int64_t n = g->n;
+    const bool mh = !jp && p.H > 1;
     r->rounds = r->inner = r->launches = 0;
     if (n == 0) return GC_OK;
     int rc = ensure_count_scratch(g);
     if (rc) return rc;
-    if (s.nbig < 0) {  // more big vertices than the shared hash set holds: witness kernel
+    if (mh && s.cnt_h < p.H) {  // H count words per vertex
+        dfree(s.cnt);
+        s.cnt = nullptr;
+        GC_CUDA_TRY(dmalloc(&s.cnt, (size_t)n * 8 * (size_t)p.H));
+        s.cnt_h = p.H;
+    }
+    if (jp && (rc = ensure_jp_scratch(g))) return rc;
+    if (GC_PACKED && s.nbig < 0) {  // more big vertices than the shared hash set holds
+        if (jp) return run_luby(g, p, r);
+        if (mh) return run_sweep_maxmin(g, p, r);
         rc = ensure_scratch(g, true, false);
         return rc ? rc : run_persistent_maxmin(g, p, r);
     }
+    // max-min colours >= 2 vertices of every uncoloured component per round;
+    // JP >= 1 (its rounds are the longest decreasing-weight path)
     const int64_t max_rounds = std::min<int64_t>(std::min<int64_t>(p.max_rounds, 0xFFFFFFF0ll),
-                                                 n / 2 + 2);
+                                                 jp ? n + 2 : mh ? std::min<int64_t>(n / 2 + 2, (1ll << 27) - 2)
+                                                             : n / 2 + 2);
     rc = ensure_nk(g, std::min<int64_t>(std::min<int64_t>(n + 2, max_rounds + 2), 1 << 20));
     if (rc) return rc;
     cudaStream_t st = g->stream;
@@ -986,8 +1310,17 @@ int run_count_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
         const int64_t warps = (n + 31) / 32;
         const int blocks = (int)std::min<int64_t>((warps + 7) / 8, (int64_t)g->sm_count * 16);
         uint2 *hubs = reinterpret_cast<uint2 *>(s.hubs);
-        k_count<<<blocks, 256, 0, st>>>(g->ro, g->ci, n, key, s.cnt, hubs, nhubs);
-        k_count_hub<<<g->sm_count * 8, 256, 0, st>>>(g->ro, g->ci, key, s.cnt, hubs, nhubs);
+        CountKeys ck;
+        ck.H = p.H;
+        for (int j = 0; j < GC_MAX_HASHES; ++j) ck.k[j] = p.keys.k[j];
+        if (mh) {
+            k_count<true><<<blocks, 256, 0, st>>>(g->ro, g->ci, n, ck, s.cnt, hubs, nhubs, 0);
+            k_count_hub<true><<<g->sm_count * 8, 256, 0, st>>>(g->ro, g->ci, ck, s.cnt, hubs, nhubs, 0);
+        } else {
+            k_count<false><<<blocks, 256, 0, st>>>(g->ro, g->ci, n, ck, s.cnt, hubs, nhubs, jp ? 1 : 0);
+            k_count_hub<false><<<g->sm_count * 8, 256, 0, st>>>(g->ro, g->ci, ck, s.cnt, hubs, nhubs,
+                                                                jp ? 1 : 0);
+        }
         GC_CUDA_TRY(cudaGetLastError());
     }
     if (prof) GC_CUDA_TRY(cudaEventRecord(e1, st));
@@ -1012,9 +1345,15 @@ int run_count_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     a.max_rounds = (uint32_t)max_rounds;
     a.sl_cap = (unsigned long long)s.sl_cap;
     a.wl_cap = (unsigned long long)s.wl_cap;
+    a.jslot = s.jslot;
+    a.jslot_cap = (unsigned long long)s.jslot_cap;
+    a.H = p.H;
+    for (int j = 0; j < GC_MAX_HASHES; ++j) a.mkeys[j] = p.keys.k[j];
     if (prof) GC_CUDA_TRY(cudaMemsetAsync(s.rstat, 0, sizeof(int64_t) * 16 * (size_t)s.nk_cap, st));
     int blocks = 0;
-    rc = prof ? launch<true>(g, a, &blocks) : launch<false>(g, a, &blocks);
+    if (jp) rc = prof ? launch<true, true, false>(g, a, &blocks) : launch<false, true, false>(g, a, &blocks);
+    else if (mh) rc = prof ? launch<true, false, true>(g, a, &blocks) : launch<false, false, true>(g, a, &blocks);
+    else rc = prof ? launch<true, false, false>(g, a, &blocks) : launch<false, false, false>(g, a, &blocks);
     if (rc) return rc;
     r->launches += 3;  // k_count, k_count_hub, persistent kernel
     if (prof) GC_CUDA_TRY(cudaEventRecord(e2, st));
@@ -1023,17 +1362,17 @@ int run_count_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     GC_CUDA_TRY(cudaStreamSynchronize(st));
     if (h[cErr] != 0) {
         char buf[200];
-        if (h[cErr] == 4)
+        if (h[cErr] == 4 || h[cErr] == 5 || h[cErr] == 7)
             snprintf(buf, sizeof(buf), "count underflow at vertex %llu in round %llu: the adjacency is "
                      "not symmetric", h[cErr + 2], h[cErr + 1]);
         else
             snprintf(buf, sizeof(buf), "internal consistency check %llu failed in round %llu (vertex %llu)",
                      h[cErr], h[cErr + 1], h[cErr + 2]);
         set_error(buf);
-        return h[cErr] == 4 ? GC_ERR_NOT_SYMMETRIC : GC_ERR_CUDA;
+        return (h[cErr] == 4 || h[cErr] == 5 || h[cErr] == 7) ? GC_ERR_NOT_SYMMETRIC : GC_ERR_CUDA;
     }
     if (h[cCol] != (unsigned long long)n) {
-        set_error("max-min colouring stalled with uncoloured vertices: the adjacency is not symmetric");
+        set_error("count-mode colouring stalled with uncoloured vertices: the adjacency is not symmetric");
         return GC_ERR_NOT_SYMMETRIC;
     }
     r->rounds = (int64_t)h[cRounds];
@@ -1068,5 +1407,8 @@ int run_count_maxmin(gc_graph *g, const RunParams &p, RunResult *r) {
     }
     return GC_OK;
 }
+
+int run_count_maxmin(gc_graph *g, const RunParams &p, RunResult *r) { return run_count(g, p, r, false); }
+int run_count_jp(gc_graph *g, const RunParams &p, RunResult *r) { return run_count(g, p, r, true); }
 
 }  // namespace gc

@@ -62,7 +62,8 @@ struct Scratch {
     int64_t bitmap_words = 0;
     int64_t *host_pinned = nullptr;  // pinned readback area
     // COUNT mode (gc_count.cu)
-    unsigned long long *cnt = nullptr;   // (hi << 32) | lo uncoloured-neighbour counts
+    unsigned long long *cnt = nullptr;   // (hi << 32) | lo uncoloured-neighbour counts (cnt_h per vertex)
+    int cnt_h = 1;
     uint32_t *cnt32 = nullptr;           // packed (hi << 16) | lo counts (degree <= 65535)
     uint32_t *big = nullptr;             // vertices of degree > 65535
     uint32_t *big32 = nullptr;           // their per-side counts and flags
@@ -73,6 +74,8 @@ struct Scratch {
     uint32_t *hubs = nullptr;            // k_count: rows counted by blocks
     unsigned long long *cctr = nullptr;  // counters of the persistent count kernel
     int64_t sl_cap = 0, wl_cap = 0;
+    uint32_t *jslot = nullptr;           // JP (Luby-MIS in COUNT mode): mex slots of long rows
+    int64_t jslot_cap = 0;
 };
 
 }  // namespace gc
@@ -191,6 +194,7 @@ int run_sweep_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int run_event_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int run_count_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
+int run_count_jp(gc_graph *g, const RunParams &p, RunResult *r);
 int run_luby(gc_graph *g, const RunParams &p, RunResult *r);
 int64_t count_colors_device(gc_graph *g, const uint32_t *C, int64_t n, bool compact,
                             uint32_t *C_inout, int64_t *launches);

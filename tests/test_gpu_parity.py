@@ -48,7 +48,20 @@ def gpu_colors(g, seed, vcode, device_out=False, **kw):
 
 
 def supported_modes(vname, H):
-    return [gcb.MODE_SWEEP] if vname == "luby" else MODES
+    return [gcb.MODE_SWEEP, gcb.MODE_COUNT] if vname == "luby" else MODES
+
+
+def jp_depth(g, seed):
+    """Longest decreasing-weight path (in vertices): the number of wavefronts
+    of the COUNT-mode Luby colouring (test-side definition)."""
+    p = O.priorities(seed, 0, g.n).astype(np.int64)
+    ro, ci = g.row_offsets.numpy(), g.col_indices.numpy().astype(np.int64)
+    depth = np.zeros(g.n, dtype=np.int64)
+    for v in np.argsort(-p, kind="stable"):
+        nb = ci[ro[v]:ro[v + 1]]
+        pred = nb[p[nb] > p[v]]
+        depth[v] = 1 + (depth[pred].max() if len(pred) else 0)
+    return int(depth.max()) if g.n else 0
 
 
 # ------------------------------------------------------------- a0 weights
@@ -120,7 +133,7 @@ def test_adversarial_shapes(mode):
     ]
     for g in cases:
         for vname, H in (("maxmin", 1), ("multihash", 4), ("luby", 1)):
-            if vname == "luby" and mode != gcb.MODE_SWEEP:
+            if vname == "luby" and mode not in (gcb.MODE_SWEEP, gcb.MODE_COUNT):
                 continue
             ref = oracle_colors(g, 11, vname, H)
             C, k, st = gpu_colors(g, 11, variant_of(vname, H), mode=mode)
@@ -233,8 +246,11 @@ def test_cfg1_grid(mode):
 def test_cfg2_er_luby_and_maxmin():
     g = G.config_graph("cfg2", device="cuda").to("cpu")
     ref, ncol, inner = O.color_luby(g, 1, with_stats=True)
-    C, k, st = gpu_colors(g, 1, gcb.LUBY_MIS)
+    C, k, st = gpu_colors(g, 1, gcb.LUBY_MIS, mode=gcb.MODE_SWEEP)
     assert (C == ref).all() and k == ncol and st.inner_iterations == inner
+    C, k, st = gpu_colors(g, 1, gcb.LUBY_MIS)  # AUTO: COUNT (wavefronts)
+    assert st.mode_used == gcb.MODE_COUNT
+    assert (C == ref).all() and k == ncol and st.rounds == jp_depth(g, 1)
     ref2, R, nk = O.color_maxmin(g, 1, with_stats=True)
     for mode in MODES:
         C, k, st = gpu_colors(g, 1, gcb.MAXMIN, mode=mode, frontier_cap=4096)
@@ -256,8 +272,10 @@ def test_rmat_s18_full_oracle():
     for mode in MODES:
         C, k, st = gpu_colors(g, 1, gcb.MAXMIN, mode=mode, frontier_cap=8192)
         assert (C == ref).all() and st.rounds == R and st.frontier_sizes == nk
-    C, k, st = gpu_colors(g, 1, gcb.LUBY_MIS)
-    assert (C == O.color_luby(g, 1)).all()
+    ref_l = O.color_luby(g, 1)
+    for mode in (gcb.MODE_SWEEP, gcb.MODE_COUNT):
+        C, k, st = gpu_colors(g, 1, gcb.LUBY_MIS, mode=mode)
+        assert (C == ref_l).all()
     C, k, st = gpu_colors(g, 1, gcb.MULTIHASH(4))
     assert (C == O.color_maxmin(g, 1, 4)).all()
 
@@ -275,6 +293,54 @@ def test_cfg4_rmat_s24_certificate():
     assert O.cert_maxmin(gh, 1, 1, C) == 0
     assert O.check_proper(gh, C) == 0
     assert k == O.count_colors(C) and k in (2 * st.rounds - 1, 2 * st.rounds)
+
+
+def test_cfg4_rmat_s24_multihash_certificate():
+    """Multi-hash H=4 (COUNT mode under AUTO) at the bench size: the O(H*m)
+    certificate checks every vertex."""
+    g = G.config_graph("cfg4", device="cuda")
+    with gcb.Graph(g.n, g.row_offsets, g.col_indices, flags=gcb.BORROW_DEVICE) as h:
+        out = torch.empty(g.n, dtype=torch.int32, device="cuda")
+        _, k, st = h.color(1, gcb.MULTIHASH(4), out, stats=True)
+    assert st.mode_used == gcb.MODE_COUNT
+    C = out.cpu().numpy().view(np.uint32)
+    gh = g.to("cpu")
+    assert O.cert_maxmin(gh, 1, 4, C) == 0
+    assert O.check_proper(gh, C) == 0
+
+
+def test_luby_count_wavefronts_and_wide_mex():
+    """COUNT-mode Luby: wavefront count = longest decreasing-weight path on
+    random graphs; cliques whose mex passes the 1024-colour slot window (the
+    rescan path) and a hub star; asymmetric input falls back to SWEEP."""
+    rng = random.Random(5)
+    for i in range(40):
+        g = G.random_graph(rng.randint(1, 400), rng.choice([0.01, 0.05, 0.3]), seed=77 + i)
+        C, k, st = gpu_colors(g, i, gcb.LUBY_MIS, mode=gcb.MODE_COUNT)
+        assert (C == O.color_luby(g, i)).all() and st.rounds == jp_depth(g, i)
+    for n in (33, 1023, 1030, 2200):
+        g = G.csr_from_lists(n, [(a, b) for a in range(n) for b in range(a + 1, n)])
+        C, k, st = gpu_colors(g, 3, gcb.LUBY_MIS, mode=gcb.MODE_COUNT)
+        # closed form of the Luby colouring (pinned equal in test_oracle.py)
+        assert (C == O.color_greedy_by_priority(g, 3)).all() and k == n and st.rounds == n
+    g = _csr_tensors(300001, [(0, i) for i in range(1, 300001)] + [(1, 2), (2, 3)])
+    C, k, st = gpu_colors(g, 2, gcb.LUBY_MIS, mode=gcb.MODE_COUNT)
+    assert (C == O.color_luby(g, 2)).all()
+
+
+def test_cfg4_rmat_s24_luby_certificate():
+    """Luby-MIS (COUNT mode) at the bench size: the mex certificate
+    (first-fit in decreasing weight order, characterises it uniquely)."""
+    g = G.config_graph("cfg4", device="cuda")
+    with gcb.Graph(g.n, g.row_offsets, g.col_indices, flags=gcb.BORROW_DEVICE) as h:
+        out = torch.empty(g.n, dtype=torch.int32, device="cuda")
+        _, k, st = h.color(1, gcb.LUBY_MIS, out, stats=True)
+    assert st.mode_used == gcb.MODE_COUNT
+    C = out.cpu().numpy().view(np.uint32)
+    gh = g.to("cpu")
+    assert O.cert_mex(gh, 1, C) == 0
+    assert O.check_proper(gh, C) == 0
+    assert k == O.count_colors(C) == int(C.max()) + 1
 
 
 # ------------------------------------------------- partitioned (row e)

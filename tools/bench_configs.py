@@ -15,7 +15,8 @@ import torch  # noqa: E402
 import graphgen as G  # noqa: E402
 import paper_conf_ipps_osamatybo19_b200 as gcb  # noqa: E402
 
-MODES = {"event": gcb.MODE_EVENT, "sweep": gcb.MODE_SWEEP, "event-multi": gcb.MODE_EVENT_MULTI}
+MODES = {"event": gcb.MODE_EVENT, "sweep": gcb.MODE_SWEEP, "event-multi": gcb.MODE_EVENT_MULTI,
+         "count": gcb.MODE_COUNT, "auto": gcb.MODE_AUTO}
 
 
 def run(name, g, variant, vname, mode="event", reps=5, warm=2, loopback=0):
@@ -40,29 +41,37 @@ def run(name, g, variant, vname, mode="event", reps=5, warm=2, loopback=0):
 def main():
     dev = "cuda"
     g1 = G.config_graph("cfg1", dev)
-    run("cfg1 grid 64x64", g1, gcb.MAXMIN, "maxmin", "event")
-    run("cfg1 grid 64x64", g1, gcb.MAXMIN, "maxmin", "sweep")
-    run("cfg1 grid 64x64", g1, gcb.LUBY_MIS, "luby", "sweep")
+    for m in ("count", "event", "sweep"):
+        run("cfg1 grid 64x64", g1, gcb.MAXMIN, "maxmin", m)
+    for m in ("count", "sweep"):
+        run("cfg1 grid 64x64", g1, gcb.LUBY_MIS, "luby", m)
     g2 = G.config_graph("cfg2", dev)
-    run("cfg2 ER 2^20 d16", g2, gcb.LUBY_MIS, "luby", "sweep")
-    run("cfg2 ER 2^20 d16", g2, gcb.MAXMIN, "maxmin", "event")
-    run("cfg2 ER 2^20 d16", g2, gcb.MAXMIN, "maxmin", "sweep")
+    for m in ("count", "sweep"):
+        run("cfg2 ER 2^20 d16", g2, gcb.LUBY_MIS, "luby", m)
+    for m in ("count", "event", "sweep"):
+        run("cfg2 ER 2^20 d16", g2, gcb.MAXMIN, "maxmin", m)
     del g2
     g3 = G.config_graph("cfg3", dev)
     for H in (1, 2, 4, 8):
         run("cfg3 mesh 128^3", g3, gcb.MULTIHASH(H), f"multihash H={H}", "sweep")
     run("cfg3 mesh 128^3", g3, gcb.MAXMIN, "maxmin", "event")
+    run("cfg3 mesh 128^3", g3, gcb.MAXMIN, "maxmin", "count")
+    run("cfg3 mesh 128^3", g3, gcb.LUBY_MIS, "luby", "count")
     del g3
     gr = G.rgg(20, seed=1, device=dev)
-    run("N1 rgg_n_2_20", gr, gcb.MAXMIN, "maxmin", "event")
-    run("N1 rgg_n_2_20", gr, gcb.LUBY_MIS, "luby", "sweep")
+    run("N1 rgg_n_2_20", gr, gcb.MAXMIN, "maxmin", "count")
+    run("N1 rgg_n_2_20", gr, gcb.MAXMIN, "maxmin", "sweep")
+    run("N1 rgg_n_2_20", gr, gcb.LUBY_MIS, "luby", "count")
     del gr
     g4 = G.config_graph("cfg4", dev)
+    run("cfg4 R-MAT s24", g4, gcb.MAXMIN, "maxmin", "count")
     run("cfg4 R-MAT s24", g4, gcb.MAXMIN, "maxmin", "event")
-    run("cfg4 R-MAT s24", g4, gcb.MAXMIN, "maxmin", "event-multi", reps=2, warm=1)
-    run("cfg4 R-MAT s24", g4, gcb.MAXMIN, "maxmin", "sweep", reps=2, warm=1)
     run("cfg4 R-MAT s24", g4, gcb.MULTIHASH(4), "multihash H=4", "sweep", reps=2, warm=1)
-    run("cfg4 R-MAT s24", g4, gcb.LUBY_MIS, "luby", "sweep", reps=2, warm=1)
+    run("cfg4 R-MAT s24", g4, gcb.LUBY_MIS, "luby", "count")
+    if os.environ.get("GC_SLOW"):
+        run("cfg4 R-MAT s24", g4, gcb.MAXMIN, "maxmin", "event-multi", reps=2, warm=1)
+        run("cfg4 R-MAT s24", g4, gcb.MAXMIN, "maxmin", "sweep", reps=2, warm=1)
+        run("cfg4 R-MAT s24", g4, gcb.LUBY_MIS, "luby", "sweep", reps=2, warm=1)
     del g4
     g5 = G.rmat(22, 16, seed=1, device=dev)
     for p in (1, 2, 4, 8):
@@ -70,7 +79,7 @@ def main():
     # G3_circuit-sized FEM stand-in (the paper's only printed runtime for this
     # path, Table II: 6.68 ms on a K40c for ~1.6M vertices / 7.7M edges)
     gm = G.mesh3d(117, 117, 117)
-    run("mesh 117^3 (G3_circuit-sized)", gm, gcb.MAXMIN, "maxmin", "event")
+    run("mesh 117^3 (G3_circuit-sized)", gm, gcb.MAXMIN, "maxmin", "count")
     run("mesh 117^3 (G3_circuit-sized)", gm, gcb.MAXMIN, "maxmin", "sweep")
 
 
