@@ -540,34 +540,79 @@ __device__ __forceinline__ void walk_mh(const CArgs &a, uint32_t v, int64_t e, i
         w[q] = (v != kNone && eq < end) ? __ldcs(a.ci + eq) : kNone;
     }
     const int H = a.H;
-    uint32_t pv[GC_MAX_HASHES];
-#pragma unroll
-    for (int j = 0; j < GC_MAX_HASHES; ++j) pv[j] = j < H ? weight_mix(v ^ a.mkeys[j]) : 0u;
     bool fresh[Q];
 #pragma unroll
-    for (int q = 0; q < Q; ++q) {
-        fresh[q] = false;
-        if (w[q] == kNone) continue;
-        ++nvis;
-        unsigned long long *cw = a.cnt + (size_t)w[q] * H;
-        unsigned long long old[GC_MAX_HASHES];
-        bool hi[GC_MAX_HASHES];
+    for (int q = 0; q < Q; ++q) fresh[q] = false;
+    if (H <= 4) {
+        // H <= 4: the atomics of 4 entries x H weights are in flight together
+        uint32_t pv[4];
 #pragma unroll
-        for (int j = 0; j < GC_MAX_HASHES; ++j) {
-            if (j < H) {
-                hi[j] = pv[j] > weight_mix(w[q] ^ a.mkeys[j]);
-                old[j] = atom_add_global(cw + j, hi[j] ? kDecHi : kDecLo);
+        for (int j = 0; j < 4; ++j) pv[j] = j < H ? weight_mix(v ^ a.mkeys[j]) : 0u;
+#pragma unroll
+        for (int q0 = 0; q0 < Q; q0 += 4) {
+            unsigned long long old[4][4];
+            bool hi[4][4];
+#pragma unroll
+            for (int qq = 0; qq < 4; ++qq) {
+                const int q = q0 + qq;
+                if (q < Q && w[q] != kNone) {
+#pragma unroll
+                    for (int j = 0; j < 4; ++j) {
+                        if (j < H) {
+                            hi[qq][j] = pv[j] > weight_mix(w[q] ^ a.mkeys[j]);
+                            old[qq][j] = atom_add_global(a.cnt + (size_t)w[q] * H + j, hi[qq][j] ? kDecHi : kDecLo);
+                        }
+                    }
+                }
+            }
+#pragma unroll
+            for (int qq = 0; qq < 4; ++qq) {
+                const int q = q0 + qq;
+                if (q < Q && w[q] != kNone) {
+                    ++nvis;
+#pragma unroll
+                    for (int j = 0; j < 4; ++j) {
+                        if (j < H) {
+                            const uint32_t side = hi[qq][j] ? (uint32_t)(old[qq][j] >> 32) : (uint32_t)old[qq][j];
+                            if (side == 1u) {
+                                const uint32_t code = ((k + 1u) << 5) | ((uint32_t)j << 1) | (hi[qq][j] ? 1u : 0u);
+                                if (atomicMin(a.Zlo + w[q], code) == kNever) fresh[q] = true;
+                            } else if (side == 0u) {
+                                flag_error(a, 4, k, w[q]);
+                            }
+                        }
+                    }
+                }
             }
         }
+    } else {
+        uint32_t pv[GC_MAX_HASHES];
 #pragma unroll
-        for (int j = 0; j < GC_MAX_HASHES; ++j) {
-            if (j < H) {
-                const uint32_t side = hi[j] ? (uint32_t)(old[j] >> 32) : (uint32_t)old[j];
-                if (side == 1u) {
-                    const uint32_t code = ((k + 1u) << 5) | ((uint32_t)j << 1) | (hi[j] ? 1u : 0u);
-                    if (atomicMin(a.Zlo + w[q], code) == kNever) fresh[q] = true;
-                } else if (side == 0u) {
-                    flag_error(a, 4, k, w[q]);
+        for (int j = 0; j < GC_MAX_HASHES; ++j) pv[j] = j < H ? weight_mix(v ^ a.mkeys[j]) : 0u;
+#pragma unroll
+        for (int q = 0; q < Q; ++q) {
+            if (w[q] == kNone) continue;
+            ++nvis;
+            unsigned long long *cw = a.cnt + (size_t)w[q] * H;
+            unsigned long long old[GC_MAX_HASHES];
+            bool hi[GC_MAX_HASHES];
+#pragma unroll
+            for (int j = 0; j < GC_MAX_HASHES; ++j) {
+                if (j < H) {
+                    hi[j] = pv[j] > weight_mix(w[q] ^ a.mkeys[j]);
+                    old[j] = atom_add_global(cw + j, hi[j] ? kDecHi : kDecLo);
+                }
+            }
+#pragma unroll
+            for (int j = 0; j < GC_MAX_HASHES; ++j) {
+                if (j < H) {
+                    const uint32_t side = hi[j] ? (uint32_t)(old[j] >> 32) : (uint32_t)old[j];
+                    if (side == 1u) {
+                        const uint32_t code = ((k + 1u) << 5) | ((uint32_t)j << 1) | (hi[j] ? 1u : 0u);
+                        if (atomicMin(a.Zlo + w[q], code) == kNever) fresh[q] = true;
+                    } else if (side == 0u) {
+                        flag_error(a, 4, k, w[q]);
+                    }
                 }
             }
         }

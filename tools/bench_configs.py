@@ -54,6 +54,7 @@ def main():
     g3 = G.config_graph("cfg3", dev)
     for H in (1, 2, 4, 8):
         run("cfg3 mesh 128^3", g3, gcb.MULTIHASH(H), f"multihash H={H}", "sweep")
+        run("cfg3 mesh 128^3", g3, gcb.MULTIHASH(H), f"multihash H={H}", "count")
     run("cfg3 mesh 128^3", g3, gcb.MAXMIN, "maxmin", "event")
     run("cfg3 mesh 128^3", g3, gcb.MAXMIN, "maxmin", "count")
     run("cfg3 mesh 128^3", g3, gcb.LUBY_MIS, "luby", "count")
@@ -66,12 +67,14 @@ def main():
     g4 = G.config_graph("cfg4", dev)
     run("cfg4 R-MAT s24", g4, gcb.MAXMIN, "maxmin", "count")
     run("cfg4 R-MAT s24", g4, gcb.MAXMIN, "maxmin", "event")
-    run("cfg4 R-MAT s24", g4, gcb.MULTIHASH(4), "multihash H=4", "sweep", reps=2, warm=1)
+    for H in (2, 4, 8):
+        run("cfg4 R-MAT s24", g4, gcb.MULTIHASH(H), f"multihash H={H}", "count")
     run("cfg4 R-MAT s24", g4, gcb.LUBY_MIS, "luby", "count")
     if os.environ.get("GC_SLOW"):
         run("cfg4 R-MAT s24", g4, gcb.MAXMIN, "maxmin", "event-multi", reps=2, warm=1)
         run("cfg4 R-MAT s24", g4, gcb.MAXMIN, "maxmin", "sweep", reps=2, warm=1)
         run("cfg4 R-MAT s24", g4, gcb.LUBY_MIS, "luby", "sweep", reps=2, warm=1)
+        run("cfg4 R-MAT s24", g4, gcb.MULTIHASH(4), "multihash H=4", "sweep", reps=2, warm=1)
     del g4
     g5 = G.rmat(22, 16, seed=1, device=dev)
     for p in (1, 2, 4, 8):
