@@ -273,6 +273,9 @@ def main():
     mode_used = {1: "sweep", 2: "event (persistent)", 3: "event (multi-kernel)",
                  4: "count (persistent)"}.get(
         st.mode_used, str(st.mode_used))
+    if world > 1:
+        mode_used = {1: "sweep", 4: "count"}.get(st.mode_used, str(st.mode_used)) + \
+            " (1D vertex ranges, per-round NCCL all-gather of coloured pairs)"
 
     # ---- roofline of the dominant kernel: a profiled pass (GC_PROFILE brackets
     # every sweep launch with events on this stream); separate from the timed steps

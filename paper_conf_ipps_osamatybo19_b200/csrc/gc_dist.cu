@@ -22,47 +22,11 @@
 #include <cstring>
 #include <vector>
 
-#include "gc_internal.cuh"
-
-#ifdef GC_HAVE_NCCL
-#include <nccl.h>
-#endif
+#include "gc_dist.cuh"
 
 namespace gc {
 
 int fill_u32(uint32_t *p, uint32_t val, int64_t n, cudaStream_t st);
-
-struct Part {
-    int64_t v0 = 0, v1 = 0, nnz = 0;
-    int64_t *ro = nullptr;  // local offsets (start at 0)
-    uint32_t *ci = nullptr; // global column ids
-    bool owns_ro = false;
-    uint32_t *C = nullptr;  // replicated colours [n_global]
-    uint32_t *F[2] = {nullptr, nullptr};
-    uint32_t *hub = nullptr;
-    uint2 *colored = nullptr;  // pairs coloured this round [cap]
-    uint2 *recv = nullptr;     // world * cap pairs
-    unsigned long long *ctr = nullptr;
-    unsigned long long *cnt_send = nullptr;  // [2]: coloured, remaining
-    unsigned long long *cnt_recv = nullptr;  // [2 * world]
-    int64_t *nk = nullptr;
-    int64_t nk_cap = 1;
-};
-
-struct Dist {
-    int64_t n_global = 0;
-    int world = 1;
-    int rank = 0;
-    bool loopback = false;
-    int64_t cap = 0;  // max vertices owned by any partition (pair padding)
-    std::vector<Part> parts;
-    unsigned long long *host_cnt = nullptr;  // pinned [2 * world]
-#ifdef GC_HAVE_NCCL
-    ncclComm_t comm = nullptr;
-#endif
-};
-
-namespace {
 
 int nccl_fail(int e, const char *what) {
 #ifdef GC_HAVE_NCCL
@@ -74,6 +38,8 @@ int nccl_fail(int e, const char *what) {
     set_error(m);
     return GC_ERR_NCCL;
 }
+
+namespace {
 
 __global__ void k_pack_counts(const unsigned long long *ctr, uint32_t k,
                               unsigned long long *cnt_send) {
@@ -120,6 +86,7 @@ int alloc_part(Part &p, int64_t n_global, int64_t cap, int world) {
 }
 
 void free_part(Part &p) {
+    free_dist_count(p);
     if (p.owns_ro) dfree(p.ro);
     dfree(p.C);
     dfree(p.F[0]);
@@ -156,6 +123,11 @@ int exchange(gc_graph *g, size_t bytes, SendF send, RecvF recv) {
 }
 
 }  // namespace
+
+int dist_exchange(gc_graph *g, size_t bytes, const std::vector<const void *> &send,
+                  const std::vector<void *> &recv) {
+    return exchange(g, bytes, [&](int q) { return send[q]; }, [&](int q) { return recv[q]; });
+}
 
 void destroy_dist(gc_graph *g) {
     if (!g || !g->dist) return;
@@ -433,7 +405,13 @@ int64_t gc_color_dist(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_
     RunResult res;
     int64_t *fs = stats ? stats->frontier_sizes : nullptr;
     const int64_t fcap = stats ? stats->frontier_cap : 0;
-    rc = run_dist(g, p, &res, fs, fcap);
+    // max-min: COUNT rounds (gc_dist_count.cu) unless SWEEP is asked for;
+    // multi-hash: the sweep rounds
+    const int mode_used = (H == 1 && o->mode != GC_MODE_SWEEP) ? GC_MODE_COUNT : GC_MODE_SWEEP;
+    if (mode_used == GC_MODE_COUNT)
+        rc = run_dist_count(g, p, &res, fs, fcap);
+    else
+        rc = run_dist(g, p, &res, fs, fcap);
     if (rc) {
         cudaEventDestroy(e0);
         cudaEventDestroy(e1);
@@ -468,7 +446,7 @@ int64_t gc_color_dist(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_
         return GC_ERR_TOO_LARGE;
     }
     if (stats) {
-        stats->mode_used = GC_MODE_SWEEP;
+        stats->mode_used = mode_used;
         stats->rounds = res.rounds;
         stats->inner_iterations = res.inner;
         stats->n_colors = ncol;

@@ -353,11 +353,31 @@ def test_loopback_partitions(parts):
                         (G.rmat(13, 16, seed=7), "multihash", 3),
                         (G.csr_from_lists(5, [(0, 1), (1, 2)]), "maxmin", 1)):
         ref, R, nk = O.color_maxmin(g, 9, H, with_stats=True)
+        modes = [gcb.MODE_AUTO, gcb.MODE_SWEEP] if H == 1 else [gcb.MODE_AUTO]
         with gcb.loopback_graph(g.n, g.row_offsets, g.col_indices, parts) as h:
-            out = torch.empty(g.n, dtype=torch.int32)
-            _, k, st = h.color(9, variant_of(vname, H), out, stats=True, frontier_cap=8192)
-            assert (out.numpy().view(np.uint32) == ref).all(), (parts, g.name)
-            assert st.rounds == R and st.frontier_sizes == nk and k == O.count_colors(ref)
+            for mode in modes:
+                out = torch.empty(g.n, dtype=torch.int32)
+                _, k, st = h.color(9, variant_of(vname, H), out, stats=True, frontier_cap=8192,
+                                   mode=mode)
+                assert st.mode_used == (gcb.MODE_COUNT if H == 1 and mode == gcb.MODE_AUTO
+                                        else gcb.MODE_SWEEP)
+                assert (out.numpy().view(np.uint32) == ref).all(), (parts, g.name, mode)
+                assert st.rounds == R and st.frontier_sizes == nk and k == O.count_colors(ref)
             outc = torch.empty(g.n, dtype=torch.int32)
             h.color(9, variant_of(vname, H), outc, flags=gcb.COMPACT)
             assert (outc.numpy().view(np.uint32) == O.compact_colors(ref)).all()
+
+
+@pytest.mark.parametrize("parts", [2, 8])
+def test_loopback_count_hubs_and_ghost_rows(parts):
+    """Distributed COUNT rounds on skewed graphs: hub rows longer than the
+    block-chunk threshold (own and ghost rows), a star across partitions."""
+    cases = [G.rmat(16, 16, seed=3),
+             _csr_tensors(20001, [(0, i) for i in range(1, 20001)] + [(5, 9), (9, 17)])]
+    for g in cases:
+        ref, R, nk = O.color_maxmin(g, 4, with_stats=True)
+        with gcb.loopback_graph(g.n, g.row_offsets, g.col_indices, parts) as h:
+            out = torch.empty(g.n, dtype=torch.int32)
+            _, k, st = h.color(4, gcb.MAXMIN, out, stats=True, frontier_cap=1 << 16)
+            assert (out.numpy().view(np.uint32) == ref).all()
+            assert st.rounds == R and st.frontier_sizes == nk

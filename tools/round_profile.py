@@ -79,7 +79,9 @@ def main():
             print(nm, tot, hh)
     res = {"scale": a.scale, "mode": a.mode, "rounds": R, "n_colors": k, "ms": st.ms,
            "kernel_ms": st.kernel_ms, "buckets": summ, "op_histograms": hist,
-           "top_rounds": sorted(rows, key=lambda x: -sum(x["us"]))[:25]}
+           "top_rounds": sorted(rows, key=lambda x: -sum(x["us"]))[:25],
+           "rows": [[x["k"], round(sum(x["us"]), 2)] + list(x["stats"][:4]) for x in rows]
+           if mode == gcb.MODE_COUNT else None}
     os.makedirs(os.path.dirname(a.out) or ".", exist_ok=True)
     with open(a.out, "w") as f:
         json.dump(res, f, indent=1)
