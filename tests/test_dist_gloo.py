@@ -78,3 +78,98 @@ def test_local_csr_from_pairs_matches_global():
         ro, ci = gdist.local_csr_from_pairs(3000, v0, v1, us, vs)
         ro_ref, ci_ref = gdist.local_rows(g, v0, v1)
         assert torch.equal(ro, ro_ref) and torch.equal(ci, ci_ref)
+
+
+# ----------------------------------------------------------------------------
+# The partitioned COUNT protocol (csrc/gc_dist_count.cu) as a
+# plain model over gloo, world size 2: owned counts, ghost rows, per-round
+# all-gather of coloured pairs.  Checks the protocol (what each rank must
+# know each round) against the oracle; the CUDA kernels implementing it are
+# checked bit-exactly on the GPU (loopback and NCCL tests).
+def _count_protocol_worker(rank, world, port, q, scale, seed):
+    import numpy as np
+
+    import oracle as O
+    os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        g = G.rmat(scale, 8, seed=seed)
+        n = g.n
+        v0, v1 = gdist.split_range(n, world, rank)
+        ro, ci = (t.numpy() for t in gdist.local_rows(g, v0, v1))
+        p = O.priorities(seed, 0, n).astype(np.int64)
+        nl = v1 - v0
+        hi = np.zeros(nl, dtype=np.int64)
+        lo = np.zeros(nl, dtype=np.int64)
+        ghost = {}
+        for lv in range(nl):
+            row = ci[ro[lv]:ro[lv + 1]].astype(np.int64)
+            hi[lv] = int((p[row] > p[v0 + lv]).sum())
+            lo[lv] = len(row) - hi[lv]
+            for u in row:
+                if not v0 <= u < v1:
+                    ghost.setdefault(int(u), []).append(lv)
+        UNC, NEVER = 0xFFFFFFFF, 1 << 62
+        C = np.full(n, UNC, dtype=np.uint32)
+        Z = np.full(nl, NEVER, dtype=np.int64)
+        S = [(lv, lo[lv] == 0) for lv in range(nl) if hi[lv] == 0 or lo[lv] == 0]
+        k, remaining = 0, n
+        while remaining > 0:
+            nxt = []
+
+            def dec(pv, lw):
+                nonlocal nxt
+                if pv > p[v0 + lw]:
+                    hi[lw] -= 1
+                    side, other, lo_side = hi[lw], lo[lw], False
+                else:
+                    lo[lw] -= 1
+                    side, other, lo_side = lo[lw], hi[lw], True
+                assert side >= 0
+                if side == 0:
+                    if other > 0:
+                        nxt.append((lw, lo_side))
+                    elif lo_side:
+                        Z[lw] = k + 1
+            pairs = []
+            for lv, lof in S:
+                c = 2 * k + (1 if (lof or Z[lv] <= k) else 0)
+                C[v0 + lv] = c
+                pairs.append((v0 + lv, c))
+                for u in ci[ro[lv]:ro[lv + 1]]:
+                    if v0 <= u < v1:
+                        dec(p[v0 + lv], int(u) - v0)
+            gathered = [None] * world
+            dist.all_gather_object(gathered, pairs)
+            assert sum(len(x) for x in gathered) > 0, "stall"
+            for r, prs in enumerate(gathered):
+                if r == rank:
+                    continue
+                for v, c in prs:
+                    C[v] = c
+                    for lw in ghost.get(v, ()):
+                        dec(p[v], lw)
+            remaining -= sum(len(x) for x in gathered)
+            S = nxt
+            k += 1
+        ref, R, _ = O.color_maxmin(g, seed, with_stats=True)
+        q.put((rank, bool((C == ref).all()), k == R))
+    finally:
+        dist.destroy_process_group()
+
+
+@pytest.mark.parametrize("scale,seed", [(9, 3), (10, 5)])
+def test_partitioned_count_protocol_world2(scale, seed):
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _free_port()
+    procs = [ctx.Process(target=_count_protocol_worker, args=(r, 2, port, q, scale, seed))
+             for r in range(2)]
+    for p in procs:
+        p.start()
+    res = sorted(q.get(timeout=300) for _ in procs)
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    assert all(r[1] for r in res), "replicated colours differ from the oracle"
+    assert all(r[2] for r in res), "round count differs from the oracle"
