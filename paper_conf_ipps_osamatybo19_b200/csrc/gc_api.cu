@@ -352,6 +352,7 @@ static void free_scratch(Scratch &s) {
     dfree(s.hubs);
     dfree(s.cctr);
     dfree(s.jslot);
+    dfree(s.cM);
     if (s.host_pinned) hfree(s.host_pinned);
     s = Scratch();
 }

@@ -41,6 +41,18 @@
 
 #include "gc_internal.cuh"
 
+#ifndef GC_SKIP_COLOURED
+#define GC_SKIP_COLOURED 0  // 1: walks test a status bit and skip coloured neighbours' atomics
+                            // (measured on R-MAT s24: 38.7 vs 34.9 ms -- the extra dependent
+                            // load costs more than the atomics it saves)
+#endif
+
+#ifndef GC_PREFETCH_WL
+#define GC_PREFETCH_WL 0  // 1: prefetch the column ids of next round's long-row segments into L2
+                          // (measured on R-MAT s24: 37.0 vs 35.0 ms -- the rounds are bound by
+                          // the memory system's random traffic, extra requests slow them)
+#endif
+
 #ifndef GC_PACKED
 #define GC_PACKED 0  // 1: 32-bit (hi << 16 | lo) round counts (measured 0.8 ms slower on R-MAT s24)
 #endif
@@ -127,6 +139,7 @@ struct CArgs {
     unsigned long long sl_cap, wl_cap;
     uint32_t *jslot;               // JP: mex slots of long rows (kSlotWords each)
     unsigned long long jslot_cap;
+    uint32_t *M;                   // status bits: 1 = uncoloured (max-min, multi-hash)
     int H;                         // MH: weight functions (count words v * H + j)
     uint32_t mkeys[GC_MAX_HASHES]; // MH: their keys K_j
 };
@@ -310,12 +323,17 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
         st.vis = 0;
     }
     if (threadIdx.x == 0) {
+        // both reservations in flight together (each is an L2 round trip)
+        const unsigned c0 = min(st.n[0], (unsigned)kStS), c1 = min(st.n[1], (unsigned)kStW);
+        const unsigned long long r0 = c0 ? atom_add_global(st.cnext[0], (unsigned long long)c0) : 0ull;
+        const unsigned long long r1 = c1 ? atom_add_global(st.cnext[1], (unsigned long long)c1) : 0ull;
+        st.n[0] = c0;
+        st.n[1] = c1;
+        st.base[0] = c0 ? st.nbase[0] + r0 : 0ull;
+        st.base[1] = c1 ? st.nbase[1] + r1 : 0ull;
         for (int i = 0; i < 2; ++i) {
-            const unsigned c = min(st.n[i], (unsigned)(i == 0 ? kStS : kStW));
-            st.n[i] = c;
-            st.base[i] = c ? st.nbase[i] + atom_add_global(st.cnext[i], (unsigned long long)c) : 0ull;
             const unsigned long long capg = i == 0 ? a.sl_cap : a.wl_cap;
-            if (c && st.base[i] + c > capg) {
+            if (st.n[i] && st.base[i] + st.n[i] > capg) {
                 flag_error(a, 2, 0, (unsigned)i);
                 st.n[i] = 0;
             }
@@ -397,9 +415,16 @@ __device__ __noinline__ void schedule_rows_slow(const CArgs &a, bool pred, uint3
 
 // Colour v in round k (its scheduled round): min (2k+1) if the lo side is
 // free at the start of round k, else max (2k) -- Alg.5 L37-42, R9.
+// v leaves the uncoloured set: its status bit is cleared (later walks skip
+// its count; a coloured vertex's counts no longer decide anything)
+__device__ __forceinline__ void clear_status(const CArgs &a, uint32_t v) {
+    if (GC_SKIP_COLOURED) atomicAnd(a.M + (v >> 5), ~(1u << (v & 31u)));
+}
+
 __device__ __forceinline__ void colour(const CArgs &a, uint32_t v, uint32_t lf, uint32_t k) {
     const bool lo_free = (lf & kLoSide) || a.Zlo[v] <= k;
     a.C[v] = 2u * k + (lo_free ? 1u : 0u);
+    clear_status(a, v);
 }
 
 // Walk entries e, e + stride, ... (< end, Q of them) of the row of v coloured
@@ -421,6 +446,14 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
     for (int q = 0; q < Q; ++q) {
         const int64_t eq = e + (int64_t)q * stride;
         w[q] = (v != kNone && eq < end) ? __ldcs(a.ci + eq) : kNone;
+    }
+    if (!JP && GC_SKIP_COLOURED) {  // coloured neighbours: no atomic (their counts are dead)
+        uint32_t mb[Q];
+#pragma unroll
+        for (int q = 0; q < Q; ++q) mb[q] = w[q] != kNone ? __ldcg(a.M + (w[q] >> 5)) : 0u;
+#pragma unroll
+        for (int q = 0; q < Q; ++q)
+            if (w[q] != kNone && !((mb[q] >> (w[q] & 31u)) & 1u)) w[q] = kNone;
     }
     // One atomic per entry, address and value chosen without a branch
     // (a branch around each atomic made the compiler wait for every result).
@@ -540,6 +573,14 @@ __device__ __forceinline__ void walk_mh(const CArgs &a, uint32_t v, int64_t e, i
         w[q] = (v != kNone && eq < end) ? __ldcs(a.ci + eq) : kNone;
     }
     const int H = a.H;
+    if (GC_SKIP_COLOURED) {
+        uint32_t mb[Q];
+#pragma unroll
+        for (int q = 0; q < Q; ++q) mb[q] = w[q] != kNone ? __ldcg(a.M + (w[q] >> 5)) : 0u;
+#pragma unroll
+        for (int q = 0; q < Q; ++q)
+            if (w[q] != kNone && !((mb[q] >> (w[q] & 31u)) & 1u)) w[q] = kNone;
+    }
     bool fresh[Q];
 #pragma unroll
     for (int q = 0; q < Q; ++q) fresh[q] = false;
@@ -647,6 +688,7 @@ __device__ __forceinline__ void colour_mh(const CArgs &a, uint32_t v, uint32_t k
     if ((code >> 5) != k) flag_error(a, 8, k, v);
     const uint32_t j = (code >> 1) & 15u;
     a.C[v] = 2u * (k * (uint32_t)a.H + j) + ((code & 1u) ? 0u : 1u);
+    clear_status(a, v);
 }
 
 // Whole block, end of a round: stage the items of the vertices on the fresh
@@ -733,6 +775,10 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
             si.lf = (uint32_t)min((int64_t)kSeg, (int64_t)L.len - (int64_t)q * kSeg) | ((q == 0 || JP) ? L.flags : 0u);
             if (L.dst >= 0) st.w[L.dst + q] = si;
             else a.WL[~L.dst + q] = si;
+            if (GC_PREFETCH_WL) {  // the segment walked next round: HBM -> L2 now
+                const uint32_t ln = si.lf & kLenMask;
+                for (uint32_t o = 0; o < ln; o += 32) asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ci + si.e0 + o));
+            }
         }
     }
 }
@@ -907,6 +953,11 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
             }
         }
         const unsigned word = __ballot_sync(kFull, zero);
+        if (GC_SKIP_COLOURED && !JP) {
+            // status word of these 32 vertices: uncoloured after round 0's decisions
+            const unsigned live = __ballot_sync(kFull, valid && !zero);
+            if (lane == 0) a.M[base >> 5] = live;
+        }
         if (lane == 0 && word) atomicAdd(&stage().colored, (unsigned)__popc(word));
         schedule_rows<JP>(a, zero && re > rs, v, rs, re - rs, 0u);  // walked in round 0
     }
@@ -1296,6 +1347,7 @@ int ensure_count_scratch(gc_graph *g) {
     // hub chunk list: at most nnz / kHubChunk entries
     GC_CUDA_TRY(dmalloc(&s.hubs, ((size_t)g->nnz / kHubChunk + 1) * 8));
     GC_CUDA_TRY(dmalloc(&s.cctr, kCCtrWords * sizeof(unsigned long long)));
+    GC_CUDA_TRY(dmalloc(&s.cM, (nn + 31) / 32 * 4));
     return GC_OK;
 }
 
@@ -1394,6 +1446,7 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, bool jp) {
     a.jslot_cap = (unsigned long long)s.jslot_cap;
     a.H = p.H;
     for (int j = 0; j < GC_MAX_HASHES; ++j) a.mkeys[j] = p.keys.k[j];
+    a.M = s.cM;
     if (prof) GC_CUDA_TRY(cudaMemsetAsync(s.rstat, 0, sizeof(int64_t) * 16 * (size_t)s.nk_cap, st));
     int blocks = 0;
     if (jp) rc = prof ? launch<true, true, false>(g, a, &blocks) : launch<false, true, false>(g, a, &blocks);
