@@ -50,6 +50,8 @@ def parse():
     ap.add_argument("--no-profile", action="store_true")
     ap.add_argument("--cpu-scale", type=int, default=20, help="R-MAT scale of the oracle sample")
     ap.add_argument("--quiet", action="store_true")
+    ap.add_argument("--dist", action="store_true",
+                    help="use the partitioned path even at one rank (run under torchrun)")
     return ap.parse_args()
 
 
@@ -210,7 +212,8 @@ def main():
 
     torch.cuda.set_device(local)
     dev = torch.device("cuda", local)
-    if world > 1:
+    use_dist = world > 1 or args.dist
+    if use_dist:
         dist.init_process_group("nccl", device_id=dev)
     scale = args.scale or (24 + int(round(math.log2(max(1, world)))))
     variant = {"maxmin": gcb.MAXMIN, "luby": gcb.LUBY_MIS,
@@ -219,7 +222,7 @@ def main():
             "event-multi": gcb.MODE_EVENT_MULTI, "count": gcb.MODE_COUNT}[args.mode]
 
     t0 = time.time()
-    if world > 1:
+    if use_dist:
         from paper_conf_ipps_osamatybo19_b200 import dist as gdist
         g, handle, n, nnz_global = gdist.build_partitioned_rmat(scale, 16, 1, rank, world, dev)
     else:
@@ -273,7 +276,7 @@ def main():
     mode_used = {1: "sweep", 2: "event (persistent)", 3: "event (multi-kernel)",
                  4: "count (persistent)"}.get(
         st.mode_used, str(st.mode_used))
-    if world > 1:
+    if use_dist:
         mode_used = {1: "sweep", 4: "count"}.get(st.mode_used, str(st.mode_used)) + \
             " (1D vertex ranges, per-round NCCL all-gather of coloured pairs)"
 
@@ -292,7 +295,11 @@ def main():
                  gcb.MODE_SWEEP: {0: "k_sweep", 1: "k_hub", 2: "other", 3: "other"},
                  gcb.MODE_COUNT: {0: "k_count_persistent", 1: "k_count + k_count_hub",
                                   2: "init phase (round 0)", 3: "rounds"}}[sp.mode_used]
-        if sp.mode_used in (gcb.MODE_EVENT, gcb.MODE_COUNT):
+        if use_dist:
+            names = {0: "k_dc_* round loop (COUNT, host-driven rounds + NCCL all-gathers)"
+                     if sp.mode_used == gcb.MODE_COUNT else "sweep round loop",
+                     1: "-", 2: "-", 3: "-"}
+        if sp.mode_used in (gcb.MODE_EVENT, gcb.MODE_COUNT) or use_dist:
             cls = 0  # the persistent launch; classes 2-3 (count) / 1-3 (event) are its phases
         name = names[cls]
         kms, kl, kb = sp.kernel_ms[cls], sp.kernel_launches[cls], sp.kernel_bytes[cls]
@@ -309,7 +316,7 @@ def main():
 
     # ---- end to end through the C ABI with host buffers
     e2e = None
-    if not args.no_e2e and world == 1:
+    if not args.no_e2e and not use_dist:
         ro_h = g.row_offsets.cpu().pin_memory()
         ci_h = g.col_indices.cpu().pin_memory()
         out_h = torch.empty(n, dtype=torch.int32).pin_memory()
@@ -332,6 +339,39 @@ def main():
                "d2h_bytes_per_step": 4 * n, "ms_per_step": em,
                "includes": "gc_create_csr (H2D copy + validation) + gc_color (D2H colours) + "
                            "gc_destroy, pinned host buffers"}
+    elif not args.no_e2e:
+        # every rank: its rows from pinned host memory -> gc_create_csr_dist (NCCL
+        # communicator, ghost rows) -> gc_color (all n colours D2H) -> gc_destroy
+        from paper_conf_ipps_osamatybo19_b200 import dist as gdist
+        ro_l, ci_l = g
+        v0, v1 = gdist.split_range(n, world, rank)
+        ro_h = ro_l.cpu().pin_memory()
+        ci_h = ci_l.cpu().pin_memory()
+        out_h = torch.empty(n, dtype=torch.int32).pin_memory()
+        dstream = torch.cuda.default_stream()
+        e2e_ms = []
+        for i in range(max(1, min(args.steps, 3)) + 1):
+            flush.fill_(i & 0xFF)
+            torch.cuda.synchronize()
+            barrier()
+            a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            a.record(dstream)
+            uid = gdist.broadcast_unique_id(gcb.nccl_unique_id() if rank == 0 else None)
+            with gcb.dist_graph(n, v0, v1, ro_h, ci_h, uid, rank, world) as h2:
+                h2.color(1, variant, out_h, mode=mode)
+            b.record(dstream)
+            torch.cuda.synchronize()
+            if i > 0:
+                e2e_ms.append(a.elapsed_time(b))
+        t = torch.tensor([sum(e2e_ms) / len(e2e_ms)], dtype=torch.float64, device=dev)
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        em = float(t.item())
+        e2e = {"value": nnz_global / (em / 1e3) / 1e9, "unit": UNIT,
+               "h2d_bytes_per_step": 8 * (n + world) + 4 * nnz_global,
+               "d2h_bytes_per_step": 4 * n * world, "ms_per_step": em,
+               "includes": "per rank: gc_create_csr_dist (H2D copy of its rows, NCCL "
+                           "communicator, ghost rows) + gc_color (D2H of all colours) + "
+                           "gc_destroy, pinned host buffers; max over ranks"}
 
     cpu = None
     if rank == 0 and world == 1 and not args.no_cpu_baseline:
@@ -350,7 +390,7 @@ def main():
                                         "seeded label permutation, graph seed 1",
                            "n": n, "nnz": nnz_global, "variant": args.variant, "seed": 1,
                            "mode": mode_used,
-                           "parallelism": "1 GPU" if world == 1 else f"1D vertex ranges x{world}",
+                           "parallelism": f"1D vertex ranges x{world}" if use_dist else "1 GPU",
                            "l2": "flushed before every timed colouring (256 MiB write outside "
                                  "the events); col_indices alone exceed L2"},
                 "n_colors": ncol, "rounds": rounds[-1],
@@ -359,7 +399,7 @@ def main():
                 "roofline": roof, "cpu_baseline": cpu, "e2e": e2e}
         print(json.dumps(line), flush=True)
     handle.close()
-    if world > 1:
+    if use_dist:
         dist.destroy_process_group()
 
 

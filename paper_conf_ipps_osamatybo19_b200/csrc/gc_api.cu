@@ -353,6 +353,7 @@ static void free_scratch(Scratch &s) {
     dfree(s.cctr);
     dfree(s.jslot);
     dfree(s.cM);
+    dfree(s.crow);
     if (s.host_pinned) hfree(s.host_pinned);
     s = Scratch();
 }

@@ -53,6 +53,13 @@
                           // the memory system's random traffic, extra requests slow them)
 #endif
 
+#ifndef GC_COUNT_STREAM
+#define GC_COUNT_STREAM 0  // 1: counting pass as a chunked HBM stream (k_count_stream); measured
+                           // on R-MAT s24: 1.33 ms (1.75 TB/s) vs 0.96 + 0.28 ms for the
+                           // degree-binned k_count + k_count_hub, so the binned pass stays
+#endif
+constexpr bool kCountStream = GC_COUNT_STREAM != 0;
+
 #ifndef GC_PACKED
 #define GC_PACKED 0  // 1: 32-bit (hi << 16 | lo) round counts (measured 0.8 ms slower on R-MAT s24)
 #endif
@@ -1239,6 +1246,132 @@ __global__ void __launch_bounds__(256) k_count_hub(const int64_t *__restrict__ r
     }
 }
 
+// ------------------------------------------------ streaming counting pass
+// The counting pass is the one full sweep of the CSR (it is round 0's
+// max/min test of Alg.5 for every vertex), so it is written as an HBM
+// stream: block-iterations take fixed chunks of kCE consecutive column ids
+// (8 per thread, 16-byte vector loads, fully coalesced), whatever the degree
+// mix.  The rows overlapping a chunk are found from crow[] (the row holding
+// each chunk's first entry, computed once per graph); a thread finds the row
+// of its first entry by binary search in the block's shared copy of the row
+// offsets and walks forward.  Per-row hi counts are accumulated in shared
+// memory; rows inside the chunk are written once, rows crossing a chunk
+// boundary (pre-set by k_count_zero) get one 64-bit atomic per chunk.
+constexpr int kCT = 256;            // threads per block
+constexpr int kCE = 8 * kCT;        // entries per chunk
+constexpr int kCR = 1024;           // rows per shared batch
+
+// crow[c] = last row r with ro[r] <= c * kCE (crow[0] = 0, crow[nch] = n - 1)
+__global__ void k_chunk_rows(const int64_t *__restrict__ ro, int64_t n, int64_t nch, uint32_t *crow) {
+    for (int64_t c = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; c <= nch;
+         c += (int64_t)gridDim.x * blockDim.x) {
+        if (c == 0 || c == nch) {
+            crow[c] = c == 0 ? 0u : (uint32_t)(n - 1);
+            continue;
+        }
+        const int64_t e = c * kCE;
+        int64_t lo = 0, hi = n;  // ro[lo] <= e < ro[hi]
+        while (hi - lo > 1) {
+            const int64_t mid = (lo + hi) >> 1;
+            if (ro[mid] <= e) lo = mid;
+            else hi = mid;
+        }
+        crow[c] = (uint32_t)lo;
+    }
+}
+
+// rows crossing a chunk boundary start from zero (JP: lo pinned at 1)
+__global__ void k_count_zero(const int64_t *__restrict__ ro, const uint32_t *__restrict__ crow, int64_t nch,
+                             unsigned long long *cnt, int jp) {
+    for (int64_t c = 1 + (int64_t)blockIdx.x * blockDim.x + threadIdx.x; c < nch;
+         c += (int64_t)gridDim.x * blockDim.x) {
+        const uint32_t r = crow[c];
+        if (ro[r] < c * kCE) cnt[r] = jp ? 1ull : 0ull;
+    }
+}
+
+__global__ void __launch_bounds__(kCT) k_count_stream(const int64_t *__restrict__ ro, const uint32_t *__restrict__ ci,
+                                                      int64_t m, int64_t nch, const uint32_t *__restrict__ crow,
+                                                      uint32_t key, unsigned long long *cnt, int jp) {
+    __shared__ int64_t ro_sh[kCR + 1];
+    __shared__ uint32_t h_sh[kCR];
+    for (int64_t c = blockIdx.x; c < nch; c += gridDim.x) {
+        const int64_t c0 = c * kCE, c1 = min(m, c0 + kCE);
+        const bool last_chunk = c == nch - 1;
+        const int64_t r0 = crow[c], r1 = crow[c + 1];
+        // the first batch's entries start at c0 (ro[crow[c]] <= c0): their loads
+        // go out together with the row offsets'
+        uint32_t u[8];
+        auto load_u = [&](int64_t ef, int64_t eh) {
+            if ((reinterpret_cast<uintptr_t>(ci + ef) & 15) == 0 && ef + 8 <= eh) {
+                const uint4 a0 = __ldcs(reinterpret_cast<const uint4 *>(ci + ef));
+                const uint4 a1 = __ldcs(reinterpret_cast<const uint4 *>(ci + ef + 4));
+                u[0] = a0.x; u[1] = a0.y; u[2] = a0.z; u[3] = a0.w;
+                u[4] = a1.x; u[5] = a1.y; u[6] = a1.z; u[7] = a1.w;
+            } else {
+#pragma unroll
+                for (int q = 0; q < 8; ++q) u[q] = ef + q < eh ? __ldcs(ci + ef + q) : 0u;
+            }
+        };
+        load_u(c0 + 8 * (int64_t)threadIdx.x, c1);
+        for (int64_t rb = r0; rb <= r1; rb += kCR) {
+            const int nr = (int)min((int64_t)kCR, r1 - rb + 1);
+            __syncthreads();
+            for (int i = threadIdx.x; i <= nr; i += kCT) ro_sh[i] = ro[rb + i];
+            for (int i = threadIdx.x; i < nr; i += kCT) h_sh[i] = 0u;
+            __syncthreads();
+            const int64_t e_lo = max(ro_sh[0], c0), e_hi = min(ro_sh[nr], c1);
+            const int64_t e_first = e_lo + 8 * (int64_t)threadIdx.x;
+            if (rb != r0 && e_first < e_hi) load_u(e_first, e_hi);
+            if (e_first < e_hi) {
+                // row of e_first: last i with ro_sh[i] <= e_first
+                int lo = 0, hi = nr;
+                while (hi - lo > 1) {
+                    const int mid = (lo + hi) >> 1;
+                    if (ro_sh[mid] <= e_first) lo = mid;
+                    else hi = mid;
+                }
+                int ri = lo;
+                int64_t rend = ro_sh[ri + 1];
+                uint32_t pv = weight_mix((uint32_t)(rb + ri) ^ key);
+                uint32_t acc = 0;
+#pragma unroll
+                for (int q = 0; q < 8; ++q) {
+                    const int64_t e = e_first + q;
+                    if (e < e_hi) {
+                        if (e >= rend) {
+                            if (acc) atomicAdd(&h_sh[ri], acc);
+                            acc = 0;
+                            do {
+                                ++ri;
+                                rend = ro_sh[ri + 1];
+                            } while (e >= rend);
+                            pv = weight_mix((uint32_t)(rb + ri) ^ key);
+                        }
+                        acc += weight_mix(u[q] ^ key) > pv ? 1u : 0u;
+                    }
+                }
+                if (acc) atomicAdd(&h_sh[ri], acc);
+            }
+            __syncthreads();
+            for (int i = threadIdx.x; i < nr; i += kCT) {
+                const int64_t rs = ro_sh[i], re = ro_sh[i + 1];
+                const uint32_t h = h_sh[i];
+                const bool partial = rs < c0 || re > c1;
+                if (partial) {
+                    const int64_t len = min(re, c1) - max(rs, c0);
+                    if (len > 0)
+                        atomicAdd(cnt + rb + i, ((unsigned long long)h << 32) + (jp ? 0ull : (unsigned long long)(len - h)));
+                } else if (rb + i < r1 || last_chunk) {
+                    // inside this chunk; row crow[c+1] (empty, starting at c1) is the next
+                    // chunk's first row, and the next chunk writes it
+                    cnt[rb + i] = ((unsigned long long)h << 32) | (unsigned long long)(jp ? 1 : (re - rs) - h);
+                }
+            }
+        }
+    }
+}
+
 template <bool PROF, bool JP, bool MH>
 int launch(gc_graph *g, CArgs &a, int *blocks_out) {
     int per_sm = 0;
@@ -1348,6 +1481,12 @@ int ensure_count_scratch(gc_graph *g) {
     GC_CUDA_TRY(dmalloc(&s.hubs, ((size_t)g->nnz / kHubChunk + 1) * 8));
     GC_CUDA_TRY(dmalloc(&s.cctr, kCCtrWords * sizeof(unsigned long long)));
     GC_CUDA_TRY(dmalloc(&s.cM, (nn + 31) / 32 * 4));
+    if (kCountStream) {  // streaming counting pass: the row of every chunk's first entry
+        s.nch = std::max<int64_t>(1, (g->nnz + kCE - 1) / kCE);
+        GC_CUDA_TRY(dmalloc(&s.crow, (size_t)(s.nch + 1) * 4));
+        k_chunk_rows<<<g->sm_count * 4, 256, 0, g->stream>>>(g->ro, g->n, s.nch, s.crow);
+        GC_CUDA_TRY(cudaGetLastError());
+    }
     return GC_OK;
 }
 
@@ -1413,6 +1552,11 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, bool jp) {
         if (mh) {
             k_count<true><<<blocks, 256, 0, st>>>(g->ro, g->ci, n, ck, s.cnt, hubs, nhubs, 0);
             k_count_hub<true><<<g->sm_count * 8, 256, 0, st>>>(g->ro, g->ci, ck, s.cnt, hubs, nhubs, 0);
+        } else if (kCountStream) {
+            const int64_t nch = s.nch;
+            k_count_zero<<<g->sm_count, 256, 0, st>>>(g->ro, s.crow, nch, s.cnt, jp ? 1 : 0);
+            k_count_stream<<<(int)std::min<int64_t>(nch, (int64_t)g->sm_count * 8), kCT, 0, st>>>(
+                g->ro, g->ci, g->nnz, nch, s.crow, key, s.cnt, jp ? 1 : 0);
         } else {
             k_count<false><<<blocks, 256, 0, st>>>(g->ro, g->ci, n, ck, s.cnt, hubs, nhubs, jp ? 1 : 0);
             k_count_hub<false><<<g->sm_count * 8, 256, 0, st>>>(g->ro, g->ci, ck, s.cnt, hubs, nhubs,

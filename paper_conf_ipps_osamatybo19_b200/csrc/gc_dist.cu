@@ -396,6 +396,9 @@ int64_t gc_color_dist(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_
     p.thread_deg_max = o->thread_deg_max > 0 ? o->thread_deg_max : 8;
     p.hub_deg_min = o->hub_deg_min > 0 ? o->hub_deg_min : 4096;
     p.max_rounds = (int64_t)(0x7FFFFFFFll / (2 * H)) + 1;
+    Profile prof;
+    prof.on = (o->flags & GC_PROFILE) != 0;
+    p.prof = &prof;
     int rc = ensure_scratch(g, false, false);
     if (rc) return rc;
     cudaEvent_t e0, e1;
@@ -447,6 +450,12 @@ int64_t gc_color_dist(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_
     }
     if (stats) {
         stats->mode_used = mode_used;
+        for (int c = 0; c < 4; ++c) {
+            stats->kernel_ms[c] = prof.ms[c];
+            stats->kernel_launches[c] = prof.launches[c];
+            stats->kernel_bytes[c] = prof.bytes[c];
+        }
+        stats->visits = prof.visits;
         stats->rounds = res.rounds;
         stats->inner_iterations = res.inner;
         stats->n_colors = ncol;

@@ -416,6 +416,21 @@ int run_dist_count(gc_graph *g, const RunParams &p, RunResult *r, int64_t *front
     for (auto &pt : d.parts) {
         int rc = ensure_dc(g, pt, n);
         if (rc) return rc;
+    }
+    // GC_PROFILE: class 0 = the whole round loop (counting pass included) on
+    // this rank, its algorithmic bytes: 16 B per owned vertex (offsets + count
+    // word) + 4 B per own entry for counting; per own entry walked 4 B id +
+    // 16 B count RMW when the neighbour is owned; per ghost entry 4 B + 16 B;
+    // 8 B per coloured pair sent, 8 B per pair received.
+    const bool prof = p.prof && p.prof->on;
+    cudaEvent_t pe0 = nullptr, pe1 = nullptr;
+    if (prof) {
+        GC_CUDA_TRY(cudaEventCreate(&pe0));
+        GC_CUDA_TRY(cudaEventCreate(&pe1));
+        GC_CUDA_TRY(cudaEventRecord(pe0, st));
+    }
+    for (auto &pt : d.parts) {
+        int rc = GC_OK;
         rc = fill_u32(pt.C, GC_UNC, n, st);
         if (rc) return rc;
         GC_CUDA_TRY(cudaMemsetAsync(pt.dc.ctr, 0, kDCtrWords * sizeof(unsigned long long), st));
@@ -488,6 +503,27 @@ int run_dist_count(gc_graph *g, const RunParams &p, RunResult *r, int64_t *front
     }
     r->rounds = k;
     r->inner = k;
+    if (prof) {
+        GC_CUDA_TRY(cudaEventRecord(pe1, st));
+        GC_CUDA_TRY(cudaEventSynchronize(pe1));
+        float ms = 0.f;
+        cudaEventElapsedTime(&ms, pe0, pe1);
+        cudaEventDestroy(pe0);
+        cudaEventDestroy(pe1);
+        int64_t bytes = 0, ents = 0;
+        for (auto &pt : d.parts) {
+            int64_t ncut = 0;
+            GC_CUDA_TRY(cudaMemcpy(&ncut, pt.dc.goff + n, sizeof(int64_t), cudaMemcpyDeviceToHost));
+            const int64_t nl = pt.v1 - pt.v0;
+            bytes += 16 * nl + 4 * pt.nnz + 20 * pt.nnz + 20 * ncut + 8 * nl + 8 * n;
+            ents += pt.nnz + ncut;
+        }
+        p.prof->ms[0] += ms;
+        p.prof->launches[0] += r->launches;
+        p.prof->bytes[0] += bytes;
+        p.prof->visits += ents;
+        p.prof->launch_us.push_back(1e3f * ms);
+    }
     return GC_OK;
 }
 

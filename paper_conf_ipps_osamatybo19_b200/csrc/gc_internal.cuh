@@ -75,6 +75,8 @@ struct Scratch {
     unsigned long long *cctr = nullptr;  // counters of the persistent count kernel
     int64_t sl_cap = 0, wl_cap = 0;
     uint32_t *cM = nullptr;              // COUNT mode: status bits (1 = uncoloured)
+    uint32_t *crow = nullptr;            // COUNT mode: row of each counting chunk's first entry
+    int64_t nch = 0;
     uint32_t *jslot = nullptr;           // JP (Luby-MIS in COUNT mode): mex slots of long rows
     int64_t jslot_cap = 0;
 };

@@ -381,3 +381,23 @@ def test_loopback_count_hubs_and_ghost_rows(parts):
             _, k, st = h.color(4, gcb.MAXMIN, out, stats=True, frontier_cap=1 << 16)
             assert (out.numpy().view(np.uint32) == ref).all()
             assert st.rounds == R and st.frontier_sizes == nk
+
+
+def test_cfg5_style_partitioned_rmat_s25():
+    """cfg5's check at the largest size a test affords: R-MAT s25 (1.08e9
+    entries) partitioned P = 2, 4 (loopback transport: the same COUNT rounds,
+    ghost rows and pair exchange as NCCL) equals P = 1 element by element, and
+    the P = 1 colouring passes the oracle's certificate."""
+    g = G.rmat(25, 16, seed=1, device="cuda")
+    with gcb.Graph(g.n, g.row_offsets, g.col_indices, flags=gcb.BORROW_DEVICE) as h:
+        one = torch.empty(g.n, dtype=torch.int32, device="cuda")
+        _, k1, st1 = h.color(1, gcb.MAXMIN, one, stats=True)
+    for parts in (2, 4):
+        with gcb.loopback_graph(g.n, g.row_offsets, g.col_indices, parts) as h:
+            outp = torch.empty(g.n, dtype=torch.int32, device="cuda")
+            _, kp, stp = h.color(1, gcb.MAXMIN, outp, stats=True)
+        assert stp.mode_used == gcb.MODE_COUNT
+        assert torch.equal(outp, one) and kp == k1 and stp.rounds == st1.rounds, parts
+    C = one.cpu().numpy().view(np.uint32)
+    gh = g.to("cpu")
+    assert O.cert_maxmin(gh, 1, 1, C) == 0
