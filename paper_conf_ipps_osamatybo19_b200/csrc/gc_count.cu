@@ -265,6 +265,7 @@ struct Stage {
     unsigned long long *cnext[2];   // item-count slots of the next round
     unsigned long long nbase[2];    // where the next round's items start
     unsigned long long *ccol;       // coloured-count slot of this round
+    unsigned long long rd[3];       // round top: SL / WL item counts, trap flag (thread 0 reads)
 };
 constexpr size_t kStageBytes = sizeof(Stage);
 
@@ -790,21 +791,6 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
     }
 }
 
-// Thread 0 of each block: append targets of round k (see the counter enum).
-__device__ __forceinline__ void set_targets(const CArgs &a, uint32_t k, unsigned long long sbase_next,
-                                            unsigned long long wbase_next) {
-    Stage &st = stage();
-    if (threadIdx.x == 0) {
-        const int nx = (int)((k + 1) % 3);
-        st.cnext[0] = a.ctr + cS + 16 * nx;
-        st.cnext[1] = a.ctr + cW + 16 * nx;
-        st.nbase[0] = sbase_next;
-        st.nbase[1] = wbase_next;
-        st.ccol = a.ctr + cK + 16 * (int)(k % 3);
-    }
-    __syncthreads();
-}
-
 // JP, whole warp converged: this long-row segment of v has put its
 // predecessors' colours into the warp's window `sb`; merge it into v's slot
 // and retire its entries; the segment that retires the last entry computes
@@ -988,7 +974,23 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
     for (;; ++k) {
         const unsigned long long t_round = PROF ? gtimer() : 0ull;
         const int cur = (int)(k % 3);
-        const unsigned long long ns = __ldcg(&a.ctr[cS + 16 * cur]), nw = __ldcg(&a.ctr[cW + 16 * cur]);
+        // one thread per block reads the round's counters (2,368 warps reading
+        // the same L2 line serialise in its slice) and sets the append targets
+        if (threadIdx.x == 0) {
+            Stage &st = stage();
+            const unsigned long long r_ns = __ldcg(&a.ctr[cS + 16 * cur]), r_nw = __ldcg(&a.ctr[cW + 16 * cur]);
+            st.rd[0] = r_ns;
+            st.rd[1] = r_nw;
+            st.rd[2] = __ldcg(&a.ctr[cErr]);
+            const int nx = (int)((k + 1) % 3);
+            st.cnext[0] = a.ctr + cS + 16 * nx;
+            st.cnext[1] = a.ctr + cW + 16 * nx;
+            st.nbase[0] = sl0 + r_ns;
+            st.nbase[1] = wl0 + r_nw;
+            st.ccol = a.ctr + cK + 16 * cur;
+        }
+        __syncthreads();
+        const unsigned long long ns = stage().rd[0], nw = stage().rd[1];
         if (gtid == 0) {
             if (k > 0) {
                 const int prv = (int)((k + 2) % 3);
@@ -1001,7 +1003,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
             a.ctr[cS + 16 * nxt2] = 0ull;  // slot of round k+2 (last read at round k-1's top)
             a.ctr[cW + 16 * nxt2] = 0ull;
         }
-        if (__ldcg(&a.ctr[cErr]) != 0ull) break;  // a trap fired (uniform: read after a barrier)
+        if (stage().rd[2] != 0ull) break;  // a trap fired (uniform: read after a barrier)
         if (ns == 0 && nw == 0) break;            // nothing scheduled: done
         if (k >= a.max_rounds) break;
         if (k > 0) last = k;  // every item of round k >= 1 colours (kFirst)
@@ -1010,7 +1012,6 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
             a.rstat[16 * k + 1] = (int64_t)nw;
         }
         const unsigned long long sl1 = sl0 + ns, wl1 = wl0 + nw;
-        set_targets(a, k, sl1, wl1);
         int64_t *prs = (PROF && (int64_t)k < a.nk_cap) ? a.rstat + 16 * k : nullptr;
         if (prs && threadIdx.x == 0)
             red_max(prs + 6, gtimer() - t_round);
