@@ -12,6 +12,9 @@ Parity status per function:
                       certificate, brute-force chi)
   color_luby          pinned (descending-priority greedy closed form, Python JP)
   color_greedy        pinned (Delta+1, closed forms)
+  color_is_alg2       pinned (golden, longest-decreasing-path DP, properness)
+  color_jp_alg4       pinned (golden, K_n / edgeless closed forms, first-free
+                      property per frontier, properness)
   paper-value parity  unpinned: the paper prints no colour count or worked
                       example for any variant (Fig.1b/3 unreadable).
 """
@@ -56,6 +59,8 @@ def lib():
         L.orc_color_maxmin.argtypes = [i64, P, P, u64, i32, P, P, i64, i64]
         L.orc_color_maxmin.restype = i64
         L.orc_color_luby.argtypes, L.orc_color_luby.restype = [i64, P, P, u64, P, P], i64
+        L.orc_color_is_alg2.argtypes, L.orc_color_is_alg2.restype = [i64, P, P, u64, P, P], i64
+        L.orc_color_jp_alg4.argtypes, L.orc_color_jp_alg4.restype = [i64, P, P, u64, P, P], i64
         L.orc_color_greedy.argtypes, L.orc_color_greedy.restype = [i64, P, P, P, P], i64
         L.orc_color_greedy_by_priority.argtypes = [i64, P, P, u64, P]
         L.orc_color_greedy_by_priority.restype = i64
@@ -145,6 +150,26 @@ def color_luby(g, seed: int, with_stats: bool = False):
     if with_stats:
         return C[:n], int(r), int(inner[0])
     return C[:n]
+
+
+def _alg2(fn, g, seed, with_stats):
+    n, ro, ci = _csr(g)
+    C = np.empty(max(n, 1), dtype=np.uint32)
+    rounds = np.zeros(1, dtype=np.int64)
+    r = fn(n, _pp(ro), _p(ci), seed, _pp(C), _pp(rounds))
+    if r < 0:
+        raise OracleError(f"{fn.__name__} failed: {r}")
+    return (C[:n], int(rounds[0])) if with_stats else C[:n]
+
+
+def color_is_alg2(g, seed: int, with_stats: bool = False):
+    """Max-only IS colouring, Alg.2 as written (colour = iteration)."""
+    return _alg2(lib().orc_color_is_alg2, g, seed, with_stats)
+
+
+def color_jp_alg4(g, seed: int, with_stats: bool = False):
+    """GraphBLAS Jones-Plassmann, Alg.2 with Alg.4's frontier colour."""
+    return _alg2(lib().orc_color_jp_alg4, g, seed, with_stats)
 
 
 def color_greedy(g, order=None):

@@ -209,9 +209,60 @@ def test_golden_hand_derived(row):
         C = O.color_maxmin(g, 1)
     elif variant.startswith("multihash"):
         C = O.color_maxmin(g, 1, int(variant[len("multihash"):]))
+    elif variant == "is_alg2":
+        C = O.color_is_alg2(g, 1)
+    elif variant == "jp_alg4":
+        C = O.color_jp_alg4(g, 1)
     else:
         C = O.color_luby(g, 1)
     assert C.tolist() == expect
+
+
+# ------------------------------------------------ Alg.2 / Alg.4
+def _longest_decreasing_path(g, seed):
+    # length (in vertices) of the longest strictly-decreasing-weight path
+    # ending at each vertex: DP over vertices in decreasing weight order
+    p = [O.priority(seed, 0, v) for v in range(g.n)]
+    adj = adjacency(g)
+    depth = [0] * g.n
+    for v in sorted(range(g.n), key=lambda x: -p[x]):
+        depth[v] = 1 + max((depth[u] for u in adj[v] if p[u] > p[v]), default=0)
+    return depth
+
+
+def test_is_alg2_is_longest_decreasing_path():
+    # Alg.2's colour of v = the iteration at which v is a local max among the
+    # uncoloured = (longest decreasing-weight path ending at v) - 1
+    for g in random_graphs(80, 40, seed0=11):
+        for seed in (1, 5):
+            C, R = O.color_is_alg2(g, seed, with_stats=True)
+            d = _longest_decreasing_path(g, seed)
+            assert C.tolist() == [x - 1 for x in d]
+            assert R == (max(d) if g.n else 0)
+            assert O.check_proper(g, C) == 0
+
+
+def test_jp_alg4_properties():
+    # Alg.4: proper; one colour per Alg.2 frontier; K_n -> ranks; edgeless ->
+    # all 0; each frontier's colour is absent from its coloured neighbours and
+    # every smaller colour is present among them (the first free colour)
+    for n in (1, 6, 17):
+        kn = G.csr_from_lists(n, [(a, b) for a in range(n) for b in range(a + 1, n)])
+        p = O.priorities(3, 0, n)
+        rank = {v: i for i, v in enumerate(sorted(range(n), key=lambda x: -int(p[x])))}
+        assert O.color_jp_alg4(kn, 3).tolist() == [rank[v] for v in range(n)]
+    assert O.color_jp_alg4(G.csr_from_lists(7, []), 2).tolist() == [0] * 7
+    for g in random_graphs(80, 40, seed0=23):
+        adj = adjacency(g)
+        C = O.color_jp_alg4(g, 4)
+        rounds = O.color_is_alg2(g, 4)  # iteration of each vertex
+        assert O.check_proper(g, C) == 0
+        for k in set(rounds.tolist()):
+            F = [v for v in range(g.n) if rounds[v] == k]
+            assert len({int(C[v]) for v in F}) == 1
+            used = {int(C[u]) for v in F for u in adj[v] if rounds[u] < k}
+            c = int(C[F[0]])
+            assert c not in used and all(x in used for x in range(c))
 
 
 # ------------------------------------------------ max-min / multi-hash oracle
