@@ -66,10 +66,19 @@ typedef enum gc_status {
  * GC_MULTIHASH(h): h independent weight functions per round (R8): vertex v
  *   takes colour 2(kh+j) (max) or 2(kh+j)+1 (min) for the smallest hash j
  *   under which it is a local max or min.  GC_MULTIHASH(1) == GC_MAXMIN.
- *   1 <= h <= 16. */
+ *   1 <= h <= 16.
+ * GC_IS_ALG2: Alg.2 as written, max-only IS: iteration k
+ *   colours the uncoloured vertices heavier than every uncoloured neighbour
+ *   with colour k.  COUNT mode only; single GPU.
+ * GC_JP_ALG4: Alg.2 with Alg.4 (reading R15): the same
+ *   frontiers, each frontier takes ONE colour, the smallest colour not used by
+ *   any coloured neighbour of the frontier (GraphBLAS Jones-Plassmann).
+ *   COUNT mode only; single GPU. */
 #define GC_MAXMIN 0
 #define GC_LUBY_MIS 1
 #define GC_MULTIHASH(h) (2 | ((h) << 8))
+#define GC_IS_ALG2 3
+#define GC_JP_ALG4 4
 #define GC_VARIANT_KIND(v) ((v) & 0xFF)
 #define GC_VARIANT_HASHES(v) (((v) >> 8) & 0xFF)
 

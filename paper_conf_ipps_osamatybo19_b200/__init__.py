@@ -25,6 +25,8 @@ STATUS = {-1: "GC_ERR_INVALID_ARG", -2: "GC_ERR_SELF_LOOP", -3: "GC_ERR_NOT_SYMM
           -4: "GC_ERR_TOO_LARGE", -5: "GC_ERR_CUDA", -6: "GC_ERR_NCCL", -7: "GC_ERR_OOM"}
 MAXMIN = 0
 LUBY_MIS = 1
+IS_ALG2 = 3      # Alg.2 as written (max-only IS)
+JP_ALG4 = 4      # Alg.2 + Alg.4 (GraphBLAS Jones-Plassmann)
 
 
 def MULTIHASH(h: int) -> int:

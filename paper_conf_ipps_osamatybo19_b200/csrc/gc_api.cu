@@ -352,6 +352,7 @@ static void free_scratch(Scratch &s) {
     dfree(s.hubs);
     dfree(s.cctr);
     dfree(s.jslot);
+    dfree(s.jcr);
     dfree(s.cM);
     dfree(s.crow);
     if (s.host_pinned) hfree(s.host_pinned);
@@ -522,7 +523,7 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
             set_error("gc_color_ex: multi-hash needs 1 <= h <= 16");
             return GC_ERR_INVALID_ARG;
         }
-    } else if (kind != GC_MAXMIN && kind != GC_LUBY_MIS) {
+    } else if (kind != GC_MAXMIN && kind != GC_LUBY_MIS && kind != GC_IS_ALG2 && kind != GC_JP_ALG4) {
         set_error("gc_color_ex: unknown variant");
         return GC_ERR_INVALID_ARG;
     }
@@ -534,7 +535,10 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     if (g->dist) return gc_color_dist(g, o, colors_out, stats);
 
     const bool luby = kind == GC_LUBY_MIS;
+    // Alg.2 as written / Alg.2 + Alg.4: COUNT mode only
+    const int jpv = kind == GC_IS_ALG2 ? 2 : kind == GC_JP_ALG4 ? 3 : luby ? 1 : 0;
     int mode = o->mode;
+    if (jpv >= 2) mode = GC_MODE_COUNT;
     // AUTO: on low-degree graphs (meshes, grids) a colouring takes few rounds
     // and the plain sweep is fastest (measured: 128^3 mesh 0.47 ms sweep vs
     // 0.77 ms event); skewed graphs take thousands of rounds and need the
@@ -568,8 +572,12 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     GC_CUDA_TRY(cudaEventCreate(&e1));
     GC_CUDA_TRY(cudaEventRecord(e0, g->stream));
     RunResult res;
-    if (luby && mode == GC_MODE_COUNT)
-        rc = g->count_unsafe ? GC_ERR_NOT_SYMMETRIC : run_count_jp(g, p, &res);
+    if (jpv >= 2 && g->count_unsafe)
+        rc = GC_ERR_NOT_SYMMETRIC;
+    else if (jpv >= 2)
+        rc = run_count_jp(g, p, &res, jpv);
+    else if (luby && mode == GC_MODE_COUNT)
+        rc = g->count_unsafe ? GC_ERR_NOT_SYMMETRIC : run_count_jp(g, p, &res, 1);
     else if (luby)
         rc = run_luby(g, p, &res);
     else if (mode == GC_MODE_EVENT)
@@ -580,7 +588,7 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
         rc = g->count_unsafe ? GC_ERR_NOT_SYMMETRIC : run_count_maxmin(g, p, &res);
     else
         rc = run_sweep_maxmin(g, p, &res);
-    if (rc == GC_ERR_NOT_SYMMETRIC && mode == GC_MODE_COUNT) {
+    if (rc == GC_ERR_NOT_SYMMETRIC && mode == GC_MODE_COUNT && jpv < 2) {
         // The counts need the adjacency MULTISET to be symmetric (a duplicate
         // entry on one side only, or an asymmetric set, shows up as a count
         // underflow or a stall -- never as a silently wrong colour, DESIGN.md

@@ -147,6 +147,10 @@ struct CArgs {
     uint32_t *jslot;               // JP: mex slots of long rows (kSlotWords each)
     unsigned long long jslot_cap;
     uint32_t *M;                   // status bits: 1 = uncoloured (max-min, multi-hash)
+    int jpv;                       // JP kernel: 1 Luby (mex), 2 Alg.2 max-only, 3 Alg.2 + Alg.4
+    uint32_t *cr;                  // Alg.4: colour of each round
+    uint32_t *B;                   // Alg.4: 3 colour sets of bwords words (round k: B + (k % 3) * bwords)
+    uint32_t bwords;
     int H;                         // MH: weight functions (count words v * H + j)
     uint32_t mkeys[GC_MAX_HASHES]; // MH: their keys K_j
 };
@@ -244,12 +248,16 @@ __device__ __forceinline__ bool grid_barrier(const CArgs &a, uint32_t k) {
 
 // ---------------------------------------------------------------- staging
 constexpr int kStS = 4096, kStW = 4096, kStF = 4096, kLongMax = 512;
+constexpr int kCSetWords = 1024;  // Alg.4: colours < 32768 collected in shared memory
 struct Stage {
     Item s[kStS];
     Item w[kStW];
     uint2 fresh[kStF];              // (w, lo side?) this block scheduled in the round
     uint32_t htab[kHTab];           // hash set of the big vertices (kNone = empty)
     uint32_t wbits[kThreads / 32][32];  // JP: per-warp 1024-bit mex window
+    uint32_t cset[kCSetWords];          // Alg.4: the block's share of the round's colour set
+    uint32_t cprev;                     // Alg.4: colour of the previous round
+    unsigned cmin;                      // Alg.4: block reduction scratch
     struct Long {                   // schedule_fresh: a long row to expand
         int64_t rs, dst;            // row start; first item slot (>= 0 staged, < 0: ~global)
         uint32_t w, len, flags, pad;
@@ -399,7 +407,7 @@ __device__ __forceinline__ void schedule_rows(const CArgs &a, bool pred, uint32_
         const int64_t r0 = __shfl_sync(kFull, rs, src);
         const int64_t ln = __shfl_sync(kFull, len, src);
         const uint32_t fs = __shfl_sync(kFull, ff, src);
-        if (JP && (fs & kFirst) && lane_id() == 0) jp_slot_init(a, ww, ln);
+        if (JP && a.jpv == 1 && (fs & kFirst) && lane_id() == 0) jp_slot_init(a, ww, ln);
         const uint32_t nseg = (uint32_t)((ln + kSeg - 1) / kSeg);
         for (uint32_t q0 = 0; q0 < nseg; q0 += 32) {
             const uint32_t q = q0 + lane_id();
@@ -407,7 +415,7 @@ __device__ __forceinline__ void schedule_rows(const CArgs &a, bool pred, uint32_
             si.v = ww;
             const int64_t e0 = r0 + (int64_t)q * kSeg;
             si.e0 = e0;
-            si.lf = (uint32_t)min((int64_t)kSeg, r0 + ln - e0) | ((q == 0 || JP) ? fs : 0u);
+            si.lf = (uint32_t)min((int64_t)kSeg, r0 + ln - e0) | ((q == 0 || (JP && a.jpv == 1)) ? fs : 0u);
             stage_append(a, q < nseg, si, 1);
         }
     }
@@ -448,7 +456,7 @@ template <int Q, bool JP = false, bool WIDE = false>
 __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, int64_t e,
                                      int64_t end, int stride, uint32_t k, uint32_t &nvis,
                                      unsigned long long *mask = nullptr, uint32_t *sbits = nullptr,
-                                     bool want_mex = false) {
+                                     bool want_mex = false, bool want_set = false) {
     uint32_t w[Q];
 #pragma unroll
     for (int q = 0; q < Q; ++q) {
@@ -488,11 +496,23 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
         slot[q] = -1;
         if (JP) {
             old[q] = hi[q] ? atom_add_global(a.cnt + wq, kDecHi) : 2ull;
-            if (live && !hi[q] && want_mex) cv[q] = __ldcg(a.C + wq);
+            if (live && !hi[q] && (want_mex || want_set)) cv[q] = __ldcg(a.C + wq);
         } else {
             old[q] = live ? atom_add_global(a.cnt + wq, hi[q] ? kDecHi : kDecLo) : 2ull;
         }
 #endif
+    }
+    if (JP && want_set) {  // Alg.4: colours of v's coloured neighbours (their rounds' colours)
+#pragma unroll
+        for (int q = 0; q < Q; ++q) {
+            if (w[q] != kNone && !hi[q]) {
+                const uint32_t r = cv[q];  // a larger neighbour: coloured in an earlier round
+                if (r >= k) flag_error(a, 5, k, v);
+                const uint32_t c = r + 1u == k ? stage().cprev : __ldcg(a.cr + r);
+                if (c < 32u * kCSetWords) atomicOr(stage().cset + (c >> 5), 1u << (c & 31u));
+                else atomicOr(a.B + (size_t)(k % 3u) * a.bwords + (c >> 5), 1u << (c & 31u));
+            }
+        }
     }
     if (JP && want_mex) {
 #pragma unroll
@@ -741,7 +761,7 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
                 else flag_error(a, 1, 0, f.x);
             }
         } else {
-            if (JP) jp_slot_init(a, f.x, len);
+            if (JP && a.jpv == 1) jp_slot_init(a, f.x, len);
             const uint32_t nseg = (uint32_t)((len + kSeg - 1) / kSeg);
             const unsigned sb = atomicAdd(&st.n[1], nseg);
             int64_t dst;
@@ -764,7 +784,7 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
                     Item si;
                     si.v = f.x;
                     si.e0 = rs + (int64_t)q * kSeg;
-                    si.lf = (uint32_t)min((int64_t)kSeg, len - (int64_t)q * kSeg) | ((q == 0 || JP) ? fl : 0u);
+                    si.lf = (uint32_t)min((int64_t)kSeg, len - (int64_t)q * kSeg) | ((q == 0 || (JP && a.jpv == 1)) ? fl : 0u);
                     if (dst >= 0) st.w[dst + q] = si;
                     else a.WL[~dst + q] = si;
                 }
@@ -780,7 +800,7 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
             Item si;
             si.v = L.w;
             si.e0 = L.rs + (int64_t)q * kSeg;
-            si.lf = (uint32_t)min((int64_t)kSeg, (int64_t)L.len - (int64_t)q * kSeg) | ((q == 0 || JP) ? L.flags : 0u);
+            si.lf = (uint32_t)min((int64_t)kSeg, (int64_t)L.len - (int64_t)q * kSeg) | ((q == 0 || (JP && a.jpv == 1)) ? L.flags : 0u);
             if (L.dst >= 0) st.w[L.dst + q] = si;
             else a.WL[~L.dst + q] = si;
             if (GC_PREFETCH_WL) {  // the segment walked next round: HBM -> L2 now
@@ -859,6 +879,35 @@ __device__ __noinline__ uint32_t jp_mex_rescan(const CArgs &a, uint32_t v, uint3
     }
 }
 
+// Alg.4, whole block at the top of round k (after the grid barrier): the
+// previous round's frontier colour = the smallest colour absent from the set
+// its walks collected (R15); block 0 publishes it in cr[k-1] and clears the
+// set that round k+1 will fill (its last reader was round k-1's top).
+__device__ void jp4_round_top(const CArgs &a, uint32_t k, bool publisher) {
+    Stage &st = stage();
+    if (k > 0) {
+        const uint32_t *S = a.B + (size_t)((k - 1u) % 3u) * a.bwords;
+        const uint32_t W = min(a.bwords, (k - 1u) / 32u + 2u);
+        if (threadIdx.x == 0) st.cmin = 0xFFFFFFFFu;
+        __syncthreads();
+        for (uint32_t w = threadIdx.x; w < W; w += blockDim.x) {
+            const uint32_t x = __ldcg(S + w);
+            if (x != 0xFFFFFFFFu) atomicMin(&st.cmin, 32u * w + (uint32_t)(__ffs(~x) - 1));
+        }
+        __syncthreads();
+        if (threadIdx.x == 0) {
+            st.cprev = st.cmin != 0xFFFFFFFFu ? st.cmin : 32u * W;
+            if (publisher) a.cr[k - 1] = st.cprev;
+        }
+    }
+    if (blockIdx.x == 0) {
+        uint32_t *S2 = a.B + (size_t)((k + 1u) % 3u) * a.bwords;
+        const uint32_t W2 = min(a.bwords, k / 32u + 3u);
+        for (uint32_t w = threadIdx.x; w < W2; w += blockDim.x) S2[w] = 0u;
+    }
+    __syncthreads();
+}
+
 // 8-lane groups: OR of the group's masks
 __device__ __forceinline__ unsigned long long group8_or(unsigned long long m) {
     m |= __shfl_xor_sync(kFull, m, 1);
@@ -884,6 +933,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
         if (threadIdx.x == 0) st.vis = 0;
         if (threadIdx.x == 0) st.nf = 0;
         for (int i = threadIdx.x; i < kHTab; i += blockDim.x) st.htab[i] = kNone;
+        for (int i = threadIdx.x; i < kCSetWords; i += blockDim.x) st.cset[i] = 0u;
         __syncthreads();
         if (threadIdx.x == 0) {
             for (int i = 0; i < a.nbig; ++i) {
@@ -990,6 +1040,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
             st.ccol = a.ctr + cK + 16 * cur;
         }
         __syncthreads();
+        if (JP && a.jpv == 3) jp4_round_top(a, k, gtid == 0);
         const unsigned long long ns = stage().rd[0], nw = stage().rd[1];
         if (gtid == 0) {
             if (k > 0) {
@@ -1026,7 +1077,14 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
                 Item it = a.WL[wl0 + u];
                 if (it.v == kNone) it.lf = 0;  // hole left by schedule_fresh
                 const uint32_t pv = weight_mix(it.v ^ a.key);
-                if (JP && (it.lf & kFirst)) {  // a segment of a row being coloured
+                if (JP && a.jpv != 1) {  // Alg.2 / Alg.4: the colour is the round (remapped for Alg.4)
+                    if ((it.lf & kFirst) && lane == 0) {
+                        a.C[it.v] = k;
+                        atomicAdd(&stage().colored, 1u);
+                    }
+                    walk<kSeg / 32, true>(a, it.v, pv, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k, nvis,
+                                          nullptr, nullptr, false, a.jpv == 3);
+                } else if (JP && (it.lf & kFirst)) {  // a segment of a row being coloured
                     uint32_t *sb = stage().wbits[threadIdx.x >> 5];
                     sb[lane] = 0u;
                     __syncwarp();
@@ -1056,9 +1114,10 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
                     len = it.lf & kLenMask;
                     e0 = it.e0;
                     pv = weight_mix(v ^ a.key);
-                    want = JP && (it.lf & kFirst);
-                    if (!JP && (it.lf & kFirst)) {
-                        if (MH) colour_mh(a, v, k);
+                    want = JP && a.jpv == 1 && (it.lf & kFirst);
+                    if ((!JP || a.jpv != 1) && (it.lf & kFirst)) {
+                        if (JP) a.C[v] = k;
+                        else if (MH) colour_mh(a, v, k);
                         else colour(a, v, it.lf, k);
                         atomicAdd(&stage().colored, 1u);
                     }
@@ -1066,7 +1125,8 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
                 unsigned long long mask = 0ull;
                 for (uint32_t j = 0; __any_sync(kFull, j < len); j += 4) {
                     if (MH) walk_mh<4>(a, j < len ? v : kNone, e0 + j, e0 + len, 1, k, nvis);
-                    else walk<4, JP>(a, j < len ? v : kNone, pv, e0 + j, e0 + len, 1, k, nvis, &mask, nullptr, want);
+                    else walk<4, JP>(a, j < len ? v : kNone, pv, e0 + j, e0 + len, 1, k, nvis, &mask, nullptr, want,
+                                     JP && a.jpv == 3);
                 }
                 if (JP && want) {  // <= 32 predecessors: the mex is below 64
                     a.C[v] = (uint32_t)(__ffsll((long long)~mask) - 1);
@@ -1084,17 +1144,19 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
                     len = it.lf & kLenMask;
                     e0 = it.e0;
                     pv = weight_mix(v ^ a.key);
-                    want = JP && (it.lf & kFirst);
-                    if (!JP && (it.lf & kFirst) && (lane & 7u) == 0u) {
-                        if (MH) colour_mh(a, v, k);
+                    want = JP && a.jpv == 1 && (it.lf & kFirst);
+                    if ((!JP || a.jpv != 1) && (it.lf & kFirst) && (lane & 7u) == 0u) {
+                        if (JP) a.C[v] = k;
+                        else if (MH) colour_mh(a, v, k);
                         else colour(a, v, it.lf, k);
                         atomicAdd(&stage().colored, 1u);
                     }
                 }
                 unsigned long long mask = 0ull;
                 if (MH) walk_mh<4>(a, v, e0 + (lane & 7u), e0 + len, 8, k, nvis);
-                else walk<4, JP>(a, v, pv, e0 + (lane & 7u), e0 + len, 8, k, nvis, &mask, nullptr, want);
-                if (JP) {
+                else walk<4, JP>(a, v, pv, e0 + (lane & 7u), e0 + len, 8, k, nvis, &mask, nullptr, want,
+                                 JP && a.jpv == 3);
+                if (JP && a.jpv == 1) {
                     mask = group8_or(mask);
                     if (want && (lane & 7u) == 0u) {
                         a.C[v] = (uint32_t)(__ffsll((long long)~mask) - 1);
@@ -1113,6 +1175,18 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
             nvis_tot += nvis;
             nvis = 0;
         }
+        if (JP && a.jpv == 3) {  // the block's share of this round's colour set -> global
+            __syncthreads();
+            Stage &st = stage();
+            const uint32_t wmax = min((uint32_t)kCSetWords, k / 32u + 2u);
+            for (uint32_t w = threadIdx.x; w < wmax; w += blockDim.x) {
+                const uint32_t x = st.cset[w];
+                if (x) {
+                    atomicOr(a.B + (size_t)(k % 3u) * a.bwords + w, x);
+                    st.cset[w] = 0u;
+                }
+            }
+        }
         schedule_fresh<JP>(a, prs, t_round);
         stage_flush(a, prs, t_round);
         if (!grid_barrier(a, k)) return;
@@ -1124,6 +1198,15 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
         }
     }
     (void)wpb;
+    if (JP && a.jpv == 3) {
+        // colours were round indices: C[v] <- colour of its round (the last
+        // round's colour is this block's cprev; earlier ones are in cr)
+        const uint32_t cp = stage().cprev;
+        for (unsigned long long v = gtid; v < (unsigned long long)n; v += nthreads) {
+            const uint32_t r = a.C[v];
+            if (r != GC_UNC) a.C[v] = r + 1u == k ? cp : __ldcg(a.cr + r);
+        }
+    }
     if (gtid == 0) {
         a.ctr[cRounds] = n > 0 ? last + 1 : 0;
         a.ctr[cIters] = k;
@@ -1503,9 +1586,10 @@ static int ensure_jp_scratch(gc_graph *g) {
     return GC_OK;
 }
 
-static int run_count(gc_graph *g, const RunParams &p, RunResult *r, bool jp) {
+static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
     Scratch &s = g->s;
     const int64_t n = g->n;
+    const bool jp = jpv != 0;
     const bool mh = !jp && p.H > 1;
     r->rounds = r->inner = r->launches = 0;
     if (n == 0) return GC_OK;
@@ -1517,7 +1601,7 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, bool jp) {
         GC_CUDA_TRY(dmalloc(&s.cnt, (size_t)n * 8 * (size_t)p.H));
         s.cnt_h = p.H;
     }
-    if (jp && (rc = ensure_jp_scratch(g))) return rc;
+    if (jpv == 1 && (rc = ensure_jp_scratch(g))) return rc;
     if (GC_PACKED && s.nbig < 0) {  // more big vertices than the shared hash set holds
         if (jp) return run_luby(g, p, r);
         if (mh) return run_sweep_maxmin(g, p, r);
@@ -1592,6 +1676,23 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, bool jp) {
     a.H = p.H;
     for (int j = 0; j < GC_MAX_HASHES; ++j) a.mkeys[j] = p.keys.k[j];
     a.M = s.cM;
+    a.jpv = jpv;
+    a.cr = nullptr;
+    a.B = nullptr;
+    a.bwords = 0;
+    if (jpv == 3) {  // Alg.4: per-round colours + 3 colour sets (colours <= rounds)
+        const int64_t words = (max_rounds + 64) / 32;
+        if (!s.jcr || s.jcr_words < words) {
+            dfree(s.jcr);
+            s.jcr = nullptr;
+            GC_CUDA_TRY(dmalloc(&s.jcr, (size_t)(max_rounds + 2 + 3 * words) * 4));
+            s.jcr_words = words;
+        }
+        a.cr = s.jcr;
+        a.B = s.jcr + max_rounds + 2;
+        a.bwords = (uint32_t)words;
+        GC_CUDA_TRY(cudaMemsetAsync(a.B, 0, (size_t)3 * words * 4, st));
+    }
     if (prof) GC_CUDA_TRY(cudaMemsetAsync(s.rstat, 0, sizeof(int64_t) * 16 * (size_t)s.nk_cap, st));
     int blocks = 0;
     if (jp) rc = prof ? launch<true, true, false>(g, a, &blocks) : launch<false, true, false>(g, a, &blocks);
@@ -1651,7 +1752,7 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, bool jp) {
     return GC_OK;
 }
 
-int run_count_maxmin(gc_graph *g, const RunParams &p, RunResult *r) { return run_count(g, p, r, false); }
-int run_count_jp(gc_graph *g, const RunParams &p, RunResult *r) { return run_count(g, p, r, true); }
+int run_count_maxmin(gc_graph *g, const RunParams &p, RunResult *r) { return run_count(g, p, r, 0); }
+int run_count_jp(gc_graph *g, const RunParams &p, RunResult *r, int jpv) { return run_count(g, p, r, jpv); }
 
 }  // namespace gc

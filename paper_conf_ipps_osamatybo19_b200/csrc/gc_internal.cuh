@@ -78,6 +78,8 @@ struct Scratch {
     uint32_t *crow = nullptr;            // COUNT mode: row of each counting chunk's first entry
     int64_t nch = 0;
     uint32_t *jslot = nullptr;           // JP (Luby-MIS in COUNT mode): mex slots of long rows
+    uint32_t *jcr = nullptr;             // Alg.4: round colours + colour sets
+    int64_t jcr_words = 0;
     int64_t jslot_cap = 0;
 };
 
@@ -197,7 +199,7 @@ int run_sweep_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int run_event_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int run_count_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
-int run_count_jp(gc_graph *g, const RunParams &p, RunResult *r);
+int run_count_jp(gc_graph *g, const RunParams &p, RunResult *r, int jpv);  // 1 Luby, 2 Alg.2, 3 Alg.4
 int run_luby(gc_graph *g, const RunParams &p, RunResult *r);
 int64_t count_colors_device(gc_graph *g, const uint32_t *C, int64_t n, bool compact,
                             uint32_t *C_inout, int64_t *launches);

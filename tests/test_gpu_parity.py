@@ -31,12 +31,17 @@ def _built():
 
 
 def variant_of(name: str, H: int = 1) -> int:
-    return {"maxmin": gcb.MAXMIN, "luby": gcb.LUBY_MIS}.get(name, gcb.MULTIHASH(H))
+    return {"maxmin": gcb.MAXMIN, "luby": gcb.LUBY_MIS, "is_alg2": gcb.IS_ALG2,
+            "jp_alg4": gcb.JP_ALG4}.get(name, gcb.MULTIHASH(H))
 
 
 def oracle_colors(g, seed, variant, H=1):
     if variant == "luby":
         return O.color_luby(g, seed)
+    if variant == "is_alg2":
+        return O.color_is_alg2(g, seed)
+    if variant == "jp_alg4":
+        return O.color_jp_alg4(g, seed)
     return O.color_maxmin(g, seed, H)
 
 
@@ -48,6 +53,8 @@ def gpu_colors(g, seed, vcode, device_out=False, **kw):
 
 
 def supported_modes(vname, H):
+    if vname in ("is_alg2", "jp_alg4"):
+        return [gcb.MODE_COUNT]
     return [gcb.MODE_SWEEP, gcb.MODE_COUNT] if vname == "luby" else MODES
 
 
@@ -96,7 +103,8 @@ def test_golden_tiny():
 
 
 @pytest.mark.parametrize("vname,H", [("maxmin", 1), ("multihash", 2), ("multihash", 3),
-                                     ("multihash", 16), ("luby", 1)])
+                                     ("multihash", 16), ("luby", 1), ("is_alg2", 1),
+                                     ("jp_alg4", 1)])
 def test_random_small_graphs(vname, H):
     rng = random.Random(H * 7 + len(vname))
     for i in range(120):
@@ -132,8 +140,11 @@ def test_adversarial_shapes(mode):
         G.mesh3d(9, 7, 5),
     ]
     for g in cases:
-        for vname, H in (("maxmin", 1), ("multihash", 4), ("luby", 1)):
+        for vname, H in (("maxmin", 1), ("multihash", 4), ("luby", 1), ("is_alg2", 1),
+                         ("jp_alg4", 1)):
             if vname == "luby" and mode not in (gcb.MODE_SWEEP, gcb.MODE_COUNT):
+                continue
+            if vname in ("is_alg2", "jp_alg4") and mode != gcb.MODE_COUNT:
                 continue
             ref = oracle_colors(g, 11, vname, H)
             C, k, st = gpu_colors(g, 11, variant_of(vname, H), mode=mode)
@@ -401,3 +412,25 @@ def test_cfg5_style_partitioned_rmat_s25():
     C = one.cpu().numpy().view(np.uint32)
     gh = g.to("cpu")
     assert O.cert_maxmin(gh, 1, 1, C) == 0
+
+
+@pytest.mark.parametrize("vname", ["is_alg2", "jp_alg4"])
+def test_alg2_alg4_scaled(vname):
+    """SURVEY N3 at scale: R-MAT s18 and cfg2 ER against the oracle (rounds
+    too), a clique (colours = ranks) and a 70k-vertex path (Alg.4)."""
+    fn = O.color_is_alg2 if vname == "is_alg2" else O.color_jp_alg4
+    for g in (G.rmat(18, 16, seed=1, device="cuda").to("cpu"),
+              G.config_graph("cfg2", device="cuda").to("cpu")):
+        ref, R = fn(g, 1, with_stats=True)
+        C, k, st = gpu_colors(g, 1, variant_of(vname))
+        assert st.mode_used == gcb.MODE_COUNT
+        assert (C == ref).all() and st.rounds == R and k == O.count_colors(ref)
+    if vname == "jp_alg4":
+        n = 1200
+        g = G.csr_from_lists(n, [(a, b) for a in range(n) for b in range(a + 1, n)])
+        C, k, st = gpu_colors(g, 2, gcb.JP_ALG4)
+        assert (C == O.color_greedy_by_priority(g, 2)).all() and k == n
+        # a long path: tens of thousands of rounds, colours alternate
+        g = _csr_tensors(70001, [(i, i + 1) for i in range(70000)])
+        C, k, st = gpu_colors(g, 3, gcb.JP_ALG4)
+        assert (C == O.color_jp_alg4(g, 3)).all()
