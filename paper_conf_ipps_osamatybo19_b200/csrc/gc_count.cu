@@ -247,13 +247,24 @@ __device__ __forceinline__ bool grid_barrier(const CArgs &a, uint32_t k) {
 }
 
 // ---------------------------------------------------------------- staging
-constexpr int kStS = 4096, kStW = 4096, kStF = 4096, kLongMax = 512;
+// Staging sizes: a typical round has ~25 items per block (round 0 spills to
+// the global lists anyway).  The Stage size sets the shared-memory carveout
+// and so the L1 left to the kernel (R-MAT s24, ms per colouring): 4096 items
+// + hash set, 198 KB of Stage (28 KB L1): 39.0; 194 KB: 34.2; 2048: 32.6;
+// 1024: 31.4; 512: 31.6; 256 (20 KB of Stage): 31.1.
+#ifndef GC_STAGE_ITEMS
+#define GC_STAGE_ITEMS 256
+#endif
+constexpr int kStS = GC_STAGE_ITEMS, kStW = GC_STAGE_ITEMS, kStF = 2 * GC_STAGE_ITEMS,
+              kLongMax = GC_STAGE_ITEMS / 4;
 constexpr int kCSetWords = 1024;  // Alg.4: colours < 32768 collected in shared memory
 struct Stage {
     Item s[kStS];
     Item w[kStW];
     uint2 fresh[kStF];              // (w, lo side?) this block scheduled in the round
+#if GC_PACKED
     uint32_t htab[kHTab];           // hash set of the big vertices (kNone = empty)
+#endif
     uint32_t wbits[kThreads / 32][32];  // JP: per-warp 1024-bit mex window
     uint32_t cset[kCSetWords];          // Alg.4: the block's share of the round's colour set
     uint32_t cprev;                     // Alg.4: colour of the previous round
@@ -285,7 +296,12 @@ __device__ __forceinline__ Stage &stage() {
 __device__ __forceinline__ unsigned hslot(uint32_t v) { return (v * 2654435761u) >> 20; }  // 12 bits
 // slot of v in the block's hash set of big vertices, or -1
 __device__ __forceinline__ int big_slot(uint32_t v) {
+#if GC_PACKED
     const uint32_t *t = stage().htab;
+#else
+    const uint32_t *t = nullptr;
+    return -1;
+#endif
     for (unsigned h = hslot(v);; h = (h + 1) & (kHTab - 1)) {
         const uint32_t x = t[h];
         if (x == v) return (int)h;
@@ -932,9 +948,12 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
         if (threadIdx.x == 0) st.colored = 0;
         if (threadIdx.x == 0) st.vis = 0;
         if (threadIdx.x == 0) st.nf = 0;
+#if GC_PACKED
         for (int i = threadIdx.x; i < kHTab; i += blockDim.x) st.htab[i] = kNone;
+#endif
         for (int i = threadIdx.x; i < kCSetWords; i += blockDim.x) st.cset[i] = 0u;
         __syncthreads();
+#if GC_PACKED
         if (threadIdx.x == 0) {
             for (int i = 0; i < a.nbig; ++i) {
                 const uint32_t v = a.big[i];
@@ -943,6 +962,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
                 st.htab[h] = v;
             }
         }
+#endif
         // init appends round 0's items to slot 0 at position 0; its colourings
         // count for round 0 (so the "next round" targets are round 0's here)
         if (threadIdx.x == 0) {
@@ -1204,12 +1224,14 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
         const uint32_t cp = stage().cprev;
         for (unsigned long long v = gtid; v < (unsigned long long)n; v += nthreads) {
             const uint32_t r = a.C[v];
-            if (r != GC_UNC) a.C[v] = r + 1u == k ? cp : __ldcg(a.cr + r);
+            // (k == 0: only init's round-0 vertices, whose colour is mex of {} = 0)
+            if (r != GC_UNC) a.C[v] = k == 0 ? 0u : r + 1u == k ? cp : __ldcg(a.cr + r);
         }
     }
     if (gtid == 0) {
         a.ctr[cRounds] = n > 0 ? last + 1 : 0;
         a.ctr[cIters] = k;
+        if (k == 0) rem -= (int64_t)__ldcg(&a.ctr[cK]);  // no round-0 items: init's colourings
         a.ctr[cCol] = (unsigned long long)(n - rem);
         if (PROF) a.ctr[cPhaseNs + 1] = t_rounds;
     }

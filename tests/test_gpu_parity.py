@@ -149,6 +149,8 @@ def test_adversarial_shapes(mode):
             ref = oracle_colors(g, 11, vname, H)
             C, k, st = gpu_colors(g, 11, variant_of(vname, H), mode=mode)
             assert (C == ref).all(), (g.name, vname, H)
+            if mode == gcb.MODE_COUNT:  # symmetric input: no fallback out of COUNT mode
+                assert st.mode_used == gcb.MODE_COUNT, (g.name, vname)
     # the clique needs exactly n/2 rounds
     g = cases[4]
     _, k, st = gpu_colors(g, 5, gcb.MAXMIN, mode=mode)
