@@ -249,11 +249,12 @@ __device__ __forceinline__ bool grid_barrier(const CArgs &a, uint32_t k) {
 // ---------------------------------------------------------------- staging
 // Staging sizes: a typical round has ~25 items per block (round 0 spills to
 // the global lists anyway).  The Stage size sets the shared-memory carveout
-// and so the L1 left to the kernel (R-MAT s24, ms per colouring): 4096 items
-// + hash set, 198 KB of Stage (28 KB L1): 39.0; 194 KB: 34.2; 2048: 32.6;
-// 1024: 31.4; 512: 31.6; 256 (20 KB of Stage): 31.1.
+// and so the L1 left to the kernel.  While the kernel kept a local copy of
+// its parameters (before __grid_constant__, below) L1 decided a lot (R-MAT
+// s24: 198 KB of Stage, 28 KB L1: 39.0 ms; 194 KB: 34.2; 20 KB: 31.1); with
+// the parameters read in place: 1024 items 28.6 ms, 256 items 28.7 ms.
 #ifndef GC_STAGE_ITEMS
-#define GC_STAGE_ITEMS 256
+#define GC_STAGE_ITEMS 1024
 #endif
 constexpr int kStS = GC_STAGE_ITEMS, kStW = GC_STAGE_ITEMS, kStF = 2 * GC_STAGE_ITEMS,
               kLongMax = GC_STAGE_ITEMS / 4;
@@ -671,32 +672,34 @@ __device__ __forceinline__ void walk_mh(const CArgs &a, uint32_t v, int64_t e, i
             }
         }
     } else {
-        uint32_t pv[GC_MAX_HASHES];
-#pragma unroll
-        for (int j = 0; j < GC_MAX_HASHES; ++j) pv[j] = j < H ? weight_mix(v ^ a.mkeys[j]) : 0u;
+        // H > 4: per entry, the weights in groups of 4 (4 atomics in flight)
 #pragma unroll
         for (int q = 0; q < Q; ++q) {
             if (w[q] == kNone) continue;
             ++nvis;
             unsigned long long *cw = a.cnt + (size_t)w[q] * H;
-            unsigned long long old[GC_MAX_HASHES];
-            bool hi[GC_MAX_HASHES];
+            for (int j0 = 0; j0 < H; j0 += 4) {
+                unsigned long long old[4];
+                bool hi[4];
 #pragma unroll
-            for (int j = 0; j < GC_MAX_HASHES; ++j) {
-                if (j < H) {
-                    hi[j] = pv[j] > weight_mix(w[q] ^ a.mkeys[j]);
-                    old[j] = atom_add_global(cw + j, hi[j] ? kDecHi : kDecLo);
+                for (int jj = 0; jj < 4; ++jj) {
+                    const int j = j0 + jj;
+                    if (j < H) {
+                        hi[jj] = weight_mix(v ^ a.mkeys[j]) > weight_mix(w[q] ^ a.mkeys[j]);
+                        old[jj] = atom_add_global(cw + j, hi[jj] ? kDecHi : kDecLo);
+                    }
                 }
-            }
 #pragma unroll
-            for (int j = 0; j < GC_MAX_HASHES; ++j) {
-                if (j < H) {
-                    const uint32_t side = hi[j] ? (uint32_t)(old[j] >> 32) : (uint32_t)old[j];
-                    if (side == 1u) {
-                        const uint32_t code = ((k + 1u) << 5) | ((uint32_t)j << 1) | (hi[j] ? 1u : 0u);
-                        if (atomicMin(a.Zlo + w[q], code) == kNever) fresh[q] = true;
-                    } else if (side == 0u) {
-                        flag_error(a, 4, k, w[q]);
+                for (int jj = 0; jj < 4; ++jj) {
+                    const int j = j0 + jj;
+                    if (j < H) {
+                        const uint32_t side = hi[jj] ? (uint32_t)(old[jj] >> 32) : (uint32_t)old[jj];
+                        if (side == 1u) {
+                            const uint32_t code = ((k + 1u) << 5) | ((uint32_t)j << 1) | (hi[jj] ? 1u : 0u);
+                            if (atomicMin(a.Zlo + w[q], code) == kNever) fresh[q] = true;
+                        } else if (side == 0u) {
+                            flag_error(a, 4, k, w[q]);
+                        }
                     }
                 }
             }
@@ -933,7 +936,10 @@ __device__ __forceinline__ unsigned long long group8_or(unsigned long long m) {
 }
 
 template <bool PROF, bool JP, bool MH>
-__global__ void __launch_bounds__(kThreads, 1) k_count_persistent(CArgs a) {
+// __grid_constant__: helpers take `const CArgs &`; without it the reference
+// to a kernel parameter forces a per-thread local copy of CArgs (272 B of
+// stack, every field access an LDL through L1): 31.1 -> 28.7 ms on R-MAT s24.
+__global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_constant__ CArgs a) {
     const unsigned lane = lane_id();
     const unsigned long long gtid = (unsigned long long)blockIdx.x * blockDim.x + threadIdx.x;
     const unsigned long long nthreads = (unsigned long long)gridDim.x * blockDim.x;
