@@ -73,7 +73,10 @@ namespace {
 constexpr unsigned kFull = 0xFFFFFFFFu;
 constexpr uint32_t kNone = 0xFFFFFFFFu;
 constexpr uint32_t kNever = 0xFFFFFFFFu;  // Z: side never free (yet)
-constexpr int kThreads = 512;              // one block per SM (128 registers)
+#ifndef GC_COUNT_THREADS
+#define GC_COUNT_THREADS 512
+#endif
+constexpr int kThreads = GC_COUNT_THREADS;  // one block per SM
 constexpr int kShortMax = 32;              // SL rows: one 8-lane group
 constexpr int kSeg = 256;                  // WL item: one warp, 8 entries per lane
 constexpr int kHubMin = 4096;              // k_count: longer rows by blocks
