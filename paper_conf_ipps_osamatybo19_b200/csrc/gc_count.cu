@@ -449,19 +449,12 @@ __device__ __noinline__ void schedule_rows_slow(const CArgs &a, bool pred, uint3
     schedule_rows<JP>(a, pred, w, rs, len, ff);
 }
 
-// Colour v in round k (its scheduled round): min (2k+1) if the lo side is
-// free at the start of round k, else max (2k) -- Alg.5 L37-42, R9.
 // v leaves the uncoloured set: its status bit is cleared (later walks skip
 // its count; a coloured vertex's counts no longer decide anything)
 __device__ __forceinline__ void clear_status(const CArgs &a, uint32_t v) {
     if (GC_SKIP_COLOURED) atomicAnd(a.M + (v >> 5), ~(1u << (v & 31u)));
 }
 
-__device__ __forceinline__ void colour(const CArgs &a, uint32_t v, uint32_t lf, uint32_t k) {
-    const bool lo_free = (lf & kLoSide) || a.Zlo[v] <= k;
-    a.C[v] = 2u * k + (lo_free ? 1u : 0u);
-    clear_status(a, v);
-}
 
 // Walk entries e, e + stride, ... (< end, Q of them) of the row of v coloured
 // in round k (v == kNone: idle lane; whole warp converged): decrement the
@@ -732,14 +725,25 @@ __device__ __forceinline__ void walk_mh(const CArgs &a, uint32_t v, int64_t e, i
     }
 }
 
-// MH: colour v in its scheduled round k from the decision code in Zlo[v]
-__device__ __forceinline__ void colour_mh(const CArgs &a, uint32_t v, uint32_t k) {
-    const uint32_t code = __ldcg(a.Zlo + v);
-    if ((code >> 5) != k) flag_error(a, 8, k, v);
-    const uint32_t j = (code >> 1) & 15u;
-    a.C[v] = 2u * (k * (uint32_t)a.H + j) + ((code & 1u) ? 0u : 1u);
+// The colour of v in its scheduled round k from its decision word z = Zlo[v]
+// (max-min: min 2k+1 if the lo side is free at the start of round k -- the
+// item's lo flag or a lo-freed-second stamp <= k --, else max 2k, Alg.5
+// L37-42, R9; MH: the decision code).  The word is loaded
+// when the item starts and consumed after the walk, so the walk's loads do
+// not wait for it (a round's decision words are final at its start: words
+// written during round k carry round k+1 and never change a round-k colour).
+template <bool MH>
+__device__ __forceinline__ void colour_fin(const CArgs &a, uint32_t v, uint32_t lf, uint32_t k, uint32_t z) {
+    if (MH) {
+        if ((z >> 5) != k) flag_error(a, 8, k, v);
+        a.C[v] = 2u * (k * (uint32_t)a.H + ((z >> 1) & 15u)) + ((z & 1u) ? 0u : 1u);
+    } else {
+        a.C[v] = 2u * k + (((lf & kLoSide) || z <= k) ? 1u : 0u);
+    }
     clear_status(a, v);
+    atomicAdd(&stage().colored, 1u);
 }
+
 
 // Whole block, end of a round: stage the items of the vertices on the fresh
 // list -- one THREAD per fresh vertex (row offsets in one dependent step),
@@ -1121,35 +1125,35 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                                                 nvis, nullptr, sb, true);
                     jp_segment_done(a, it.v, it.lf & kLenMask, pv, sb, k);
                 } else {
-                    if (!JP && (it.lf & kFirst) && lane == 0) {
-                        if (MH) colour_mh(a, it.v, k);
-                        else colour(a, it.v, it.lf, k);
-                        atomicAdd(&stage().colored, 1u);
-                    }
+                    const bool cl = !JP && (it.lf & kFirst) && lane == 0;
+                    const uint32_t z = cl ? __ldcg(a.Zlo + it.v) : 0u;
                     if (MH)
                         walk_mh<kSeg / 32>(a, it.v, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k, nvis);
                     else
                         walk<kSeg / 32, JP>(a, it.v, pv, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k, nvis);
+                    if (cl) colour_fin<MH>(a, it.v, it.lf, k, z);
                 }
             } else if (lane_rows) {
                 // short rows: one per lane, 4 entries per step
                 const unsigned long long idx = sl0 + 32 * (u - nw) + lane;
                 uint32_t v = kNone, len = 0, pv = 0;
                 int64_t e0 = 0;
-                bool want = false;
+                bool want = false, cl = false;
+                uint32_t lf = 0, z = 0;
                 if (idx < sl1) {
                     const Item it = a.SL[idx];
                     v = it.v;
+                    lf = it.lf;
                     len = it.lf & kLenMask;
                     e0 = it.e0;
                     pv = weight_mix(v ^ a.key);
                     want = JP && a.jpv == 1 && (it.lf & kFirst);
-                    if ((!JP || a.jpv != 1) && (it.lf & kFirst)) {
-                        if (JP) a.C[v] = k;
-                        else if (MH) colour_mh(a, v, k);
-                        else colour(a, v, it.lf, k);
+                    if (JP && a.jpv != 1 && (it.lf & kFirst)) {
+                        a.C[v] = k;
                         atomicAdd(&stage().colored, 1u);
                     }
+                    cl = !JP && (it.lf & kFirst);
+                    if (cl) z = __ldcg(a.Zlo + v);
                 }
                 unsigned long long mask = 0ull;
                 for (uint32_t j = 0; __any_sync(kFull, j < len); j += 4) {
@@ -1157,6 +1161,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                     else walk<4, JP>(a, j < len ? v : kNone, pv, e0 + j, e0 + len, 1, k, nvis, &mask, nullptr, want,
                                      JP && a.jpv == 3);
                 }
+                if (cl) colour_fin<MH>(a, v, lf, k, z);
                 if (JP && want) {  // <= 32 predecessors: the mex is below 64
                     a.C[v] = (uint32_t)(__ffsll((long long)~mask) - 1);
                     atomicAdd(&stage().colored, 1u);
@@ -1166,25 +1171,28 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                 const unsigned long long idx = sl0 + 4 * (u - nw) + (lane >> 3);
                 uint32_t v = kNone, len = 0, pv = 0;
                 int64_t e0 = 0;
-                bool want = false;
+                bool want = false, cl = false;
+                uint32_t lf = 0, z = 0;
                 if (idx < sl1) {
                     const Item it = a.SL[idx];
                     v = it.v;
+                    lf = it.lf;
                     len = it.lf & kLenMask;
                     e0 = it.e0;
                     pv = weight_mix(v ^ a.key);
                     want = JP && a.jpv == 1 && (it.lf & kFirst);
-                    if ((!JP || a.jpv != 1) && (it.lf & kFirst) && (lane & 7u) == 0u) {
-                        if (JP) a.C[v] = k;
-                        else if (MH) colour_mh(a, v, k);
-                        else colour(a, v, it.lf, k);
+                    if (JP && a.jpv != 1 && (it.lf & kFirst) && (lane & 7u) == 0u) {
+                        a.C[v] = k;
                         atomicAdd(&stage().colored, 1u);
                     }
+                    cl = !JP && (it.lf & kFirst) && (lane & 7u) == 0u;
+                    if (cl) z = __ldcg(a.Zlo + v);
                 }
                 unsigned long long mask = 0ull;
                 if (MH) walk_mh<4>(a, v, e0 + (lane & 7u), e0 + len, 8, k, nvis);
                 else walk<4, JP>(a, v, pv, e0 + (lane & 7u), e0 + len, 8, k, nvis, &mask, nullptr, want,
                                  JP && a.jpv == 3);
+                if (cl) colour_fin<MH>(a, v, lf, k, z);
                 if (JP && a.jpv == 1) {
                     mask = group8_or(mask);
                     if (want && (lane & 7u) == 0u) {
