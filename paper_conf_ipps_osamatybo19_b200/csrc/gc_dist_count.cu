@@ -39,7 +39,7 @@ constexpr int64_t kChunk = 1024;
 constexpr unsigned long long kDecHi = 0ull - (1ull << 32);
 constexpr unsigned long long kDecLo = ~0ull;
 
-enum : int { cSEnd = 0, cLo, cHi, cPairs, cLong, cErr, cErrV, cChunks, kDCtrWords = 16 };
+enum : int { cSEnd = 0, cLo, cHi, cPairs, cLong, cErr, cErrV, cChunks, cTicket, kDCtrWords = 16 };
 
 struct LongJob {
     int64_t s, e;     // entry range
@@ -215,17 +215,35 @@ __global__ void k_dc_count_fin(DCArgs a) {
 }
 
 // round bookkeeping: the next round's slice of S; clear the per-round counters
-__global__ void k_dc_advance(DCArgs a) {
+__device__ __forceinline__ void dc_advance(const DCArgs &a) {
     a.ctr[cLo] = a.ctr[cHi];
     a.ctr[cHi] = a.ctr[cSEnd];
     a.ctr[cPairs] = 0ull;
     a.ctr[cLong] = 0ull;
     a.ctr[cChunks] = 0ull;
 }
+__global__ void k_dc_advance(DCArgs a) { dc_advance(a); }
+
+// whole block, end of a kernel: true in one thread of the block that finishes
+// last (every block's writes and atomics are visible to it)
+__device__ __forceinline__ bool last_block(const DCArgs &a) {
+    __shared__ int last;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence();
+        last = atomicAdd(a.ctr + cTicket, 1ull) == gridDim.x - 1;
+        if (last) {
+            a.ctr[cTicket] = 0ull;
+            __threadfence();
+        }
+    }
+    __syncthreads();
+    return threadIdx.x == 0 && last;
+}
 
 // ---------------------------------------------------------------- rounds
 // 1. the owned vertices scheduled for round k: 8-lane groups
-__global__ void k_dc_walk(DCArgs a) {
+__global__ void k_dc_walk(DCArgs a, unsigned long long *cnt_send) {
     const unsigned lane = lane_id();
     const int64_t gid = ((int64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 3;
     const int64_t ng = ((int64_t)gridDim.x * blockDim.x) >> 3;
@@ -246,11 +264,10 @@ __global__ void k_dc_walk(DCArgs a) {
         }
         if (re - rs <= kLongMin) walk_entries<false>(a, weight_mix(vg ^ a.key), rs, re, sub, 8);
     }
-}
-
-__global__ void k_dc_pack(DCArgs a, unsigned long long *cnt_send) {
-    cnt_send[0] = a.ctr[cPairs];
-    cnt_send[1] = a.ctr[cErr];
+    if (last_block(a)) {  // what the all-gather of this round sends: (pairs, error flag)
+        cnt_send[0] = __ldcg(a.ctr + cPairs);
+        cnt_send[1] = __ldcg(a.ctr + cErr);
+    }
 }
 
 // 3. remote pairs: apply to C, walk the ghost rows (8-lane groups; long
@@ -291,6 +308,7 @@ __global__ void k_dc_long(DCArgs a) {
         if (L.ghost) walk_entries<true>(a, pv, c0, c1, threadIdx.x, blockDim.x);
         else walk_entries<false>(a, pv, c0, c1, threadIdx.x, blockDim.x);
     }
+    if (last_block(a)) dc_advance(a);  // the round is complete on this rank
 }
 
 // ---------------------------------------------------------------- ghost rows
@@ -461,9 +479,8 @@ int run_dist_count(gc_graph *g, const RunParams &p, RunResult *r, int64_t *front
         if (frontier && k < fcap) frontier[k] = remaining;
         for (auto &pt : d.parts) {
             DCArgs a = args_of(g, pt, key, (uint32_t)k);
-            k_dc_walk<<<blocks, 256, 0, st>>>(a);
-            k_dc_pack<<<1, 1, 0, st>>>(a, pt.cnt_send);
-            r->launches += 2;
+            k_dc_walk<<<blocks, 256, 0, st>>>(a, pt.cnt_send);
+            r->launches += 1;
         }
         int rc = dist_exchange(g, 2 * sizeof(unsigned long long), cs, cr);
         if (rc) return rc;
@@ -494,8 +511,7 @@ int run_dist_count(gc_graph *g, const RunParams &p, RunResult *r, int64_t *front
             const int self = d.loopback ? (int)q : d.rank;
             k_dc_ghost<<<blocks, 256, 0, st>>>(a, pt.recv, pt.cnt_recv, d.world, self, (int64_t)maxc);
             k_dc_long<<<blocks, 256, 0, st>>>(a);
-            k_dc_advance<<<1, 1, 0, st>>>(a);
-            r->launches += 3;
+            r->launches += 2;
         }
         GC_CUDA_TRY(cudaGetLastError());
         remaining -= (int64_t)tot;
