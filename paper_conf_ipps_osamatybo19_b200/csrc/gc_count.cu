@@ -111,11 +111,11 @@ struct __align__(16) Item {
 // that slot was round k-1's top, which every block has passed (a reader and
 // a writer of one slot are always separated by a grid barrier).
 enum : int {
-    cS = 0,         // [0, 16, 32]: SL items of the round
-    cW = 48,        // [48, 64, 80]: WL items of the round
+    cS = 0,         // [0, 16, 32]: the round words R (SL items | WL items | barrier arrivals)
+    cW = 48,        // [48, 64, 80]: (unused)
     cK = 96,        // [96, 112, 128]: vertices coloured in the round (stats)
     cCol = 144,     // vertices coloured (written at the end, host check)
-    cBar = 160,     // barrier arrivals (monotone)
+    cBar = 160,     // (unused: arrivals live in the round words)
     cAbort = 176,
     cErr = 192,     // [192..194] first trap: kind, round, vertex
     cRounds = 208,  // result: rounds R
@@ -217,20 +217,36 @@ __device__ __forceinline__ uint32_t atom_add_global32(uint32_t *p, uint32_t x) {
     return old;
 }
 
-// Grid barrier (cooperative launch: every block is resident): monotone
-// arrival counter, release arrival, acquire spin (which also invalidates the
-// SM's L1, so the next phase sees what other SMs wrote).  A wait beyond 4 s
-// records a trap and makes every block leave instead of hanging the GPU.
-__device__ __forceinline__ bool grid_barrier(const CArgs &a, uint32_t k) {
+// Round word R (one per round, 3 rotating slots): SL item count in bits
+// [0, 29), WL item count in [29, 53), barrier arrivals in [53, 64).  A block
+// reserves its items of the next round with ONE atomic (both list bases come
+// back), and the spin that ends the round's barrier reads the next round's
+// item counts in the same load that sees the last arrival.
+constexpr unsigned long long kRwWL = 1ull << 29, kRwArr = 1ull << 53;
+constexpr unsigned long long kMSL = kRwWL - 1ull, kMWL = (1ull << 24) - 1ull;
+__device__ __forceinline__ unsigned long long rw_field(unsigned long long v, int li) {
+    return li == 0 ? (v & kMSL) : ((v >> 29) & kMWL);
+}
+__device__ __forceinline__ unsigned long long rw_add(unsigned long long c, int li) {
+    return li == 0 ? c : c << 29;
+}
+
+// Grid barrier on the round word rw (all blocks resident, cooperative
+// launch): release arrival, acquire spin (which also invalidates the SM's
+// L1, so the next phase sees what other SMs wrote); thread 0 leaves the final
+// word in *out.  A wait beyond 4 s records a trap and makes every block leave
+// instead of hanging the GPU.
+__device__ __forceinline__ bool grid_barrier_rw(const CArgs &a, uint32_t k, unsigned long long *rw,
+                                                unsigned long long *out) {
     __shared__ int ok_sh;
     __syncthreads();
     if (threadIdx.x == 0) {
         int ok = 1;
-        const unsigned long long old = atom_add_release(a.ctr + cBar, 1ull);
-        const unsigned long long target = (old / gridDim.x + 1) * gridDim.x;
+        atom_add_release(rw, kRwArr);
         unsigned spins = 0;
         const unsigned long long t0 = gtimer();
-        while (ld_acquire(a.ctr + cBar) < target) {
+        unsigned long long v;
+        while (((v = ld_acquire(rw)) >> 53) < gridDim.x) {
             if ((++spins & 255u) == 0u) {
                 if (*(volatile unsigned long long *)(a.ctr + cAbort)) {
                     ok = 0;
@@ -244,11 +260,13 @@ __device__ __forceinline__ bool grid_barrier(const CArgs &a, uint32_t k) {
                 }
             }
         }
+        *out = v;
         ok_sh = ok;
     }
     __syncthreads();
     return ok_sh != 0;
 }
+
 
 // ---------------------------------------------------------------- staging
 // Staging sizes: a typical round has ~25 items per block (round 0 spills to
@@ -286,10 +304,10 @@ struct Stage {
     unsigned long long t_fs;        // PROF: when this block's fresh step started
     unsigned long long base[2];
     // append targets of the current round (set by thread 0 at the round top)
-    unsigned long long *cnext[2];   // item-count slots of the next round
+    unsigned long long *rw;         // the next round's word R (item reservations, arrivals)
     unsigned long long nbase[2];    // where the next round's items start
     unsigned long long *ccol;       // coloured-count slot of this round
-    unsigned long long rd[3];       // round top: SL / WL item counts, trap flag (thread 0 reads)
+    unsigned long long rd[4];       // round word from the barrier; SL / WL item counts, trap flag
 };
 constexpr size_t kStageBytes = sizeof(Stage);
 
@@ -303,15 +321,15 @@ __device__ __forceinline__ unsigned hslot(uint32_t v) { return (v * 2654435761u)
 __device__ __forceinline__ int big_slot(uint32_t v) {
 #if GC_PACKED
     const uint32_t *t = stage().htab;
-#else
-    const uint32_t *t = nullptr;
-    return -1;
-#endif
     for (unsigned h = hslot(v);; h = (h + 1) & (kHTab - 1)) {
         const uint32_t x = t[h];
         if (x == v) return (int)h;
         if (x == kNone) return -1;
     }
+#else
+    (void)v;
+    return -1;
+#endif
 }
 
 // Whole warp converged: lanes with `pred` append `val` to staged list li;
@@ -334,7 +352,7 @@ __device__ __forceinline__ void stage_append(const CArgs &a, bool pred, const It
     if (sm) {
         const unsigned sl = __ffs(sm) - 1;
         unsigned long long gb = 0;
-        if (lane == sl) gb = atom_add_global(st.cnext[li], (unsigned long long)__popc(sm));
+        if (lane == sl) gb = rw_field(atom_add_global(st.rw, rw_add((unsigned long long)__popc(sm), li)), li);
         gb = __shfl_sync(kFull, gb, sl);
         if (spill) {
             const unsigned long long at = st.nbase[li] + gb + __popc(sm & ((1u << lane) - 1u));
@@ -362,8 +380,10 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
     if (threadIdx.x == 0) {
         // both reservations in flight together (each is an L2 round trip)
         const unsigned c0 = min(st.n[0], (unsigned)kStS), c1 = min(st.n[1], (unsigned)kStW);
-        const unsigned long long r0 = c0 ? atom_add_global(st.cnext[0], (unsigned long long)c0) : 0ull;
-        const unsigned long long r1 = c1 ? atom_add_global(st.cnext[1], (unsigned long long)c1) : 0ull;
+        // one reservation for both lists
+        const unsigned long long rv = (c0 || c1) ? atom_add_global(st.rw, rw_add(c0, 0) + rw_add(c1, 1)) : 0ull;
+        const unsigned long long r0 = rw_field(rv, 0), r1 = rw_field(rv, 1);
+        if (r0 + c0 > kMSL || r1 + c1 > kMWL) flag_error(a, 9, 0, 0);  // a round word field overflowed
         st.n[0] = c0;
         st.n[1] = c1;
         st.base[0] = c0 ? st.nbase[0] + r0 : 0ull;
@@ -783,7 +803,7 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
             if (pos < (unsigned)kStS) {
                 st.s[pos] = it;
             } else {
-                const unsigned long long at = st.nbase[0] + atom_add_global(st.cnext[0], 1ull);
+                const unsigned long long at = st.nbase[0] + rw_field(atom_add_global(st.rw, 1ull), 0);
                 if (at < a.sl_cap) a.SL[at] = it;
                 else flag_error(a, 1, 0, f.x);
             }
@@ -797,7 +817,7 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
             } else {
                 // does not fit: global slots; staged slots [sb, kStW) become holes
                 for (unsigned h = sb; h < (unsigned)kStW && h < sb + nseg; ++h) st.w[h].v = kNone;
-                dst = ~(int64_t)(st.nbase[1] + atom_add_global(st.cnext[1], (unsigned long long)nseg));
+                dst = ~(int64_t)(st.nbase[1] + rw_field(atom_add_global(st.rw, rw_add(nseg, 1)), 1));
             }
             const unsigned li = atomicAdd(&st.nlong, 1u);
             if (li < (unsigned)kLongMax) {
@@ -980,8 +1000,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
         // init appends round 0's items to slot 0 at position 0; its colourings
         // count for round 0 (so the "next round" targets are round 0's here)
         if (threadIdx.x == 0) {
-            st.cnext[0] = a.ctr + cS;
-            st.cnext[1] = a.ctr + cW;
+            st.rw = a.ctr + cS;  // round 0's word
             st.nbase[0] = st.nbase[1] = 0ull;
             st.ccol = a.ctr + cK;
         }
@@ -1039,7 +1058,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
         schedule_rows<JP>(a, zero && re > rs, v, rs, re - rs, 0u);  // walked in round 0
     }
     stage_flush(a);
-    if (!grid_barrier(a, 0)) return;
+    if (!grid_barrier_rw(a, 0, a.ctr + cS, &stage().rd[0])) return;
     if (PROF && gtid == 0) {
         const unsigned long long t = gtimer();
         a.ctr[cPhaseNs] = t - t0;
@@ -1060,35 +1079,27 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
         const int cur = (int)(k % 3);
         // one thread per block reads the round's counters (2,368 warps reading
         // the same L2 line serialise in its slice) and sets the append targets
+        // the round's item counts came with the barrier's last load (round
+        // word); the trap flag is read every 32 rounds (a trap ends the
+        // kernel at most 32 rounds later, grid-uniformly)
         if (threadIdx.x == 0) {
             Stage &st = stage();
-            const unsigned long long r_ns = __ldcg(&a.ctr[cS + 16 * cur]), r_nw = __ldcg(&a.ctr[cW + 16 * cur]);
-            st.rd[0] = r_ns;
-            st.rd[1] = r_nw;
-            st.rd[2] = __ldcg(&a.ctr[cErr]);
-            const int nx = (int)((k + 1) % 3);
-            st.cnext[0] = a.ctr + cS + 16 * nx;
-            st.cnext[1] = a.ctr + cW + 16 * nx;
+            const unsigned long long w = st.rd[0];
+            const unsigned long long r_ns = rw_field(w, 0), r_nw = rw_field(w, 1);
+            st.rd[1] = r_ns;
+            st.rd[2] = r_nw;
+            st.rd[3] = (k & 31u) == 0u ? __ldcg(&a.ctr[cErr]) : 0ull;
+            st.rw = a.ctr + cS + 16 * (int)((k + 1) % 3);
             st.nbase[0] = sl0 + r_ns;
             st.nbase[1] = wl0 + r_nw;
             st.ccol = a.ctr + cK + 16 * cur;
         }
         __syncthreads();
         if (JP && a.jpv == 3) jp4_round_top(a, k, gtid == 0);
-        const unsigned long long ns = stage().rd[0], nw = stage().rd[1];
-        if (gtid == 0) {
-            if (k > 0) {
-                const int prv = (int)((k + 2) % 3);
-                rem -= (int64_t)__ldcg(&a.ctr[cK + 16 * prv]);
-                a.ctr[cK + 16 * prv] = 0ull;  // only gtid 0 reads these slots
-            }
-            if ((int64_t)k < a.nk_cap) a.nk[k] = rem;
-            if (PROF && k > 0 && (int64_t)(k - 1) < a.nk_cap) a.rstat[16 * (k - 1) + 3] = a.nk[k - 1] - rem;
-            const int nxt2 = (int)((k + 2) % 3);
-            a.ctr[cS + 16 * nxt2] = 0ull;  // slot of round k+2 (last read at round k-1's top)
-            a.ctr[cW + 16 * nxt2] = 0ull;
-        }
-        if (stage().rd[2] != 0ull) break;  // a trap fired (uniform: read after a barrier)
+        const unsigned long long ns = stage().rd[1], nw = stage().rd[2];
+        // word of round k+2 (its last reader: the barrier that ended round k-2)
+        if (gtid == 0) a.ctr[cS + 16 * (int)((k + 2) % 3)] = 0ull;
+        if (stage().rd[3] != 0ull) break;  // a trap fired (uniform: read after a barrier)
         if (ns == 0 && nw == 0) break;            // nothing scheduled: done
         if (k >= a.max_rounds) break;
         if (k > 0) last = k;  // every item of round k >= 1 colours (kFirst)
@@ -1213,6 +1224,15 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
             nvis_tot += nvis;
             nvis = 0;
         }
+        if (gtid == 0) {  // bookkeeping: uncoloured at the start of round k (off the round top)
+            if (k > 0) {
+                const int prv = (int)((k + 2) % 3);
+                rem -= (int64_t)__ldcg(&a.ctr[cK + 16 * prv]);
+                a.ctr[cK + 16 * prv] = 0ull;  // only gtid 0 reads these slots
+            }
+            if ((int64_t)k < a.nk_cap) a.nk[k] = rem;
+            if (PROF && k > 0 && (int64_t)(k - 1) < a.nk_cap) a.rstat[16 * (k - 1) + 3] = a.nk[k - 1] - rem;
+        }
         if (JP && a.jpv == 3) {  // the block's share of this round's colour set -> global
             __syncthreads();
             Stage &st = stage();
@@ -1227,7 +1247,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
         }
         schedule_fresh<JP>(a, prs, t_round);
         stage_flush(a, prs, t_round);
-        if (!grid_barrier(a, k)) return;
+        if (!grid_barrier_rw(a, k, a.ctr + cS + 16 * (int)((k + 1) % 3), &stage().rd[0])) return;
         if (PROF && gtid == 0) {
             const unsigned long long t = gtimer();
             if ((int64_t)k < a.nk_cap) a.rstat[16 * k + 4] = (int64_t)(t - t0);
@@ -1249,7 +1269,8 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
     if (gtid == 0) {
         a.ctr[cRounds] = n > 0 ? last + 1 : 0;
         a.ctr[cIters] = k;
-        if (k == 0) rem -= (int64_t)__ldcg(&a.ctr[cK]);  // no round-0 items: init's colourings
+        // the colourings of round k-1 (init's for k == 0) not yet subtracted
+        rem -= (int64_t)__ldcg(&a.ctr[cK + 16 * (k == 0 ? 0 : (int)((k + 2) % 3))]);
         a.ctr[cCol] = (unsigned long long)(n - rem);
         if (PROF) a.ctr[cPhaseNs + 1] = t_rounds;
     }
@@ -1508,6 +1529,10 @@ int launch(gc_graph *g, CArgs &a, int *blocks_out) {
         return GC_ERR_CUDA;
     }
     const int blocks = per_sm * g->sm_count;
+    if (blocks >= 2048) {  // the round word's arrival field has 11 bits
+        set_error("persistent count kernel: too many blocks for the round word");
+        return GC_ERR_CUDA;
+    }
     // L2 persistence for the count words (every round's decrements are a
     // burst of random 8-byte atomics; a burst that misses L2 is several times
     // slower, tools/microbench_atomics.cu).  Per-launch attribute: no stream
