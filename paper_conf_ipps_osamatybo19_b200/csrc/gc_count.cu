@@ -60,10 +60,6 @@
 #endif
 constexpr bool kCountStream = GC_COUNT_STREAM != 0;
 
-#ifndef GC_FRESH_RO
-#define GC_FRESH_RO 1  // the walk that frees a vertex loads its row offsets (not the block's fresh step)
-#endif
-
 #ifndef GC_PACKED
 #define GC_PACKED 0  // 1: 32-bit (hi << 16 | lo) round counts -- max-min only (no JP / multi-hash branch);
                      // measured 27.9 vs 28.1 ms on R-MAT s24, not worth the restriction
@@ -289,9 +285,6 @@ struct Stage {
     Item s[kStS];
     Item w[kStW];
     uint2 fresh[kStF];              // (w, lo side?) this block scheduled in the round
-#if GC_FRESH_RO
-    longlong2 fro[kStF];            // ... and their row offsets (ro[w], ro[w+1])
-#endif
 #if GC_PACKED
     uint32_t htab[kHTab];           // hash set of the big vertices (kNone = empty)
 #endif
@@ -599,37 +592,16 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
     // rows are fetched once per block at the end of the round (schedule_fresh)
     // instead of one dependent load per q here
     bool ovf[Q];
-#if GC_FRESH_RO
-    // the freed vertices' row offsets: loads issued together, consumed when
-    // they are staged (this warp's tail, overlapping the other warps' work)
-    long long frs[Q], fre[Q];
-#pragma unroll
-    for (int q = 0; q < Q; ++q) {
-        frs[q] = fre[q] = 0;
-        if (fresh[q]) {
-            frs[q] = a.ro[w[q]];
-            fre[q] = a.ro[w[q] + 1];
-        }
-    }
-#endif
 #pragma unroll
     for (int q = 0; q < Q; ++q) {
         ovf[q] = false;
         if (fresh[q]) {
-#if !GC_FRESH_RO
             // its row offsets are loaded at the end of the round: start the
             // HBM -> L2 transfer now
             asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ro + w[q]));
-#endif
             const unsigned pos = atomicAdd(&stage().nf, 1u);
-            if (pos < (unsigned)kStF) {
-                stage().fresh[pos] = make_uint2(w[q], hi[q] ? 0u : kLoSide);
-#if GC_FRESH_RO
-                stage().fro[pos] = make_longlong2(frs[q], fre[q]);
-#endif
-            } else {
-                ovf[q] = true;
-            }
+            if (pos < (unsigned)kStF) stage().fresh[pos] = make_uint2(w[q], hi[q] ? 0u : kLoSide);
+            else ovf[q] = true;
         }
     }
 #pragma unroll
@@ -755,20 +727,10 @@ __device__ __forceinline__ void walk_mh(const CArgs &a, uint32_t v, int64_t e, i
     for (int q = 0; q < Q; ++q) {
         ovf[q] = false;
         if (fresh[q]) {
-#if GC_FRESH_RO
-            const long long r0 = a.ro[w[q]], r1 = a.ro[w[q] + 1];
-#else
             asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ro + w[q]));
-#endif
             const unsigned pos = atomicAdd(&stage().nf, 1u);
-            if (pos < (unsigned)kStF) {
-                stage().fresh[pos] = make_uint2(w[q], 0u);
-#if GC_FRESH_RO
-                stage().fro[pos] = make_longlong2(r0, r1);
-#endif
-            } else {
-                ovf[q] = true;
-            }
+            if (pos < (unsigned)kStF) stage().fresh[pos] = make_uint2(w[q], 0u);
+            else ovf[q] = true;
         }
     }
 #pragma unroll
@@ -825,11 +787,7 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
     const unsigned nf = min(st.nf, (unsigned)kStF);
     for (unsigned t = threadIdx.x; t < nf; t += blockDim.x) {
         const uint2 f = st.fresh[t];
-#if GC_FRESH_RO
-        const int64_t rs = st.fro[t].x, re = st.fro[t].y;
-#else
         const int64_t rs = a.ro[f.x], re = a.ro[f.x + 1];
-#endif
         const int64_t len = re - rs;
         const uint32_t fl = kFirst | f.y;
         if (len <= kShortMax) {
