@@ -97,7 +97,8 @@ typedef enum gc_status {
 
 /* Sweep strategy (gc_options.mode).  All modes return identical colours. */
 #define GC_MODE_AUTO 0   /* max-min and multi-hash: SWEEP if max degree <= 8
-                            (meshes), else COUNT; Luby-MIS: COUNT */
+                            and n >= 2^20 (large meshes), else COUNT;
+                            Luby-MIS: COUNT */
 #define GC_MODE_SWEEP 1  /* every round re-scans each uncoloured vertex's row
                             with early exit (the paper's ComputeOp shape) */
 #define GC_MODE_EVENT 2  /* work-efficient: per-vertex witnesses + resume

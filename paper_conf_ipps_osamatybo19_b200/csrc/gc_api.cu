@@ -546,10 +546,12 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     // Luby-MIS: SWEEP runs Alg.2 + Alg.3 literally; COUNT computes the same
     // colouring (first-fit greedy in decreasing weight order, R10) as a
     // Jones-Plassmann wavefront over predecessor counts -- AUTO takes it.
-    // Measured (profiles/r01_configs.jsonl): COUNT wins on ER (0.79 vs 1.83 ms),
-    // rgg (0.66 vs 1.31) and R-MAT (35.6 vs 1689); the plain sweep only on
-    // meshes (128^3: 0.47 vs 0.57), whose rounds are few and uniform.
-    if (mode == GC_MODE_AUTO) mode = (luby || g->max_deg > 8) ? GC_MODE_COUNT : GC_MODE_SWEEP;
+    // Measured (profiles/r01_configs.jsonl): COUNT wins on ER (0.73 vs 1.83 ms),
+    // rgg (0.63 vs 1.33), R-MAT (26.8 vs 1689) and small grids (64^2: 0.10 vs
+    // 0.18, one launch); the plain sweep only on large meshes (128^3: 0.48 vs
+    // 0.58; 117^3: 0.43 vs 0.47), whose few uniform rounds stream the CSR.
+    if (mode == GC_MODE_AUTO)
+        mode = (luby || g->max_deg > 8 || g->n < (1 << 20)) ? GC_MODE_COUNT : GC_MODE_SWEEP;
     if (luby && mode != GC_MODE_COUNT) mode = GC_MODE_SWEEP;
     if (H != 1 && mode != GC_MODE_COUNT) mode = GC_MODE_SWEEP;  // multi-hash: SWEEP or COUNT
 
