@@ -574,27 +574,34 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     GC_CUDA_TRY(cudaEventCreate(&e1));
     GC_CUDA_TRY(cudaEventRecord(e0, g->stream));
     RunResult res;
-    if (jpv >= 2 && g->count_unsafe)
-        rc = GC_ERR_NOT_SYMMETRIC;
-    else if (jpv >= 2)
-        rc = run_count_jp(g, p, &res, jpv);
-    else if (luby && mode == GC_MODE_COUNT)
-        rc = g->count_unsafe ? GC_ERR_NOT_SYMMETRIC : run_count_jp(g, p, &res, 1);
+    auto run_count_variant = [&]() {
+        if (g->count_unsafe) return (int)GC_ERR_NOT_SYMMETRIC;
+        if (jpv >= 1) return run_count_jp(g, p, &res, jpv);
+        return run_count_maxmin(g, p, &res);
+    };
+    if (mode == GC_MODE_COUNT)
+        rc = run_count_variant();
     else if (luby)
         rc = run_luby(g, p, &res);
     else if (mode == GC_MODE_EVENT)
         rc = run_persistent_maxmin(g, p, &res);
     else if (mode == GC_MODE_EVENT_MULTI)
         rc = run_event_maxmin(g, p, &res);
-    else if (mode == GC_MODE_COUNT)
-        rc = g->count_unsafe ? GC_ERR_NOT_SYMMETRIC : run_count_maxmin(g, p, &res);
     else
         rc = run_sweep_maxmin(g, p, &res);
+    if (rc == GC_ERR_NOT_SYMMETRIC && mode == GC_MODE_COUNT && !g->deduped && !g->count_unsafe) {
+        // The counts need a symmetric adjacency MULTISET; duplicate entries are
+        // legal input (adjacency sets decide the colouring).  Switch the handle
+        // once to its deduplicated, row-sorted copy and rerun (gc_dedup.cu).
+        g->deduped = true;
+        rc = dedup_csr(g);
+        if (!rc) rc = run_count_variant();
+    }
     if (rc == GC_ERR_NOT_SYMMETRIC && mode == GC_MODE_COUNT && jpv < 2) {
-        // The counts need the adjacency MULTISET to be symmetric (a duplicate
-        // entry on one side only, or an asymmetric set, shows up as a count
-        // underflow or a stall -- never as a silently wrong colour, DESIGN.md
-        // 7.0).  The witness kernel only needs the adjacency set: rerun there.
+        // Still asymmetric after deduplication: the adjacency SETS are not
+        // symmetric (a count underflow or a stall -- never a silently wrong
+        // colour).  The witness / sweep kernels test the set
+        // they are given: rerun there (Alg.2 / Alg.4 have no such fallback).
         g->count_unsafe = true;
         if (luby) {
             mode = GC_MODE_SWEEP;

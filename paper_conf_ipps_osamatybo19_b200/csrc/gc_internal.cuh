@@ -99,7 +99,8 @@ struct gc_graph {
     gc::Scratch s;
     gc::Dist *dist = nullptr;
     int sm_count = 148;
-    bool count_unsafe = false;  // COUNT mode saw an asymmetric multiset: use EVENT
+    bool count_unsafe = false;  // COUNT mode saw an asymmetric adjacency SET: use EVENT / SWEEP
+    bool deduped = false;       // ro / ci were replaced by their deduplicated copy (gc_dedup.cu)
 };
 
 namespace gc {
@@ -199,6 +200,7 @@ int run_sweep_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int run_event_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int run_count_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
+int dedup_csr(gc_graph *g);  // gc_dedup.cu
 int run_count_jp(gc_graph *g, const RunParams &p, RunResult *r, int jpv);  // 1 Luby, 2 Alg.2, 3 Alg.4
 int run_luby(gc_graph *g, const RunParams &p, RunResult *r);
 int64_t count_colors_device(gc_graph *g, const uint32_t *C, int64_t n, bool compact,

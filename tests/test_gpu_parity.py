@@ -175,10 +175,16 @@ def test_duplicates_and_unsorted_rows():
     g2 = G.Graph(g.n, torch.tensor(nro, dtype=torch.int64),
                  torch.tensor([x for r in rows for x in r], dtype=torch.int32))
     for mode in MODES:
-        C, _, _ = gpu_colors(g2, 9, gcb.MAXMIN, mode=mode)
+        C, _, st = gpu_colors(g2, 9, gcb.MAXMIN, mode=mode)
         assert (C == ref).all()
-    C, _, _ = gpu_colors(g2, 9, gcb.LUBY_MIS)
-    assert (C == O.color_luby(g, 9)).all()
+        if mode == gcb.MODE_COUNT:  # one-sided duplicates: the deduplicated copy, still COUNT
+            assert st.mode_used == gcb.MODE_COUNT
+    for vname in ("luby", "is_alg2", "jp_alg4"):
+        C, _, st = gpu_colors(g2, 9, variant_of(vname))
+        assert (C == oracle_colors(g, 9, vname)).all(), vname
+        assert st.mode_used == gcb.MODE_COUNT
+    C, _, st = gpu_colors(g2, 9, gcb.MULTIHASH(3), mode=gcb.MODE_COUNT)
+    assert (C == O.color_maxmin(g, 9, 3)).all() and st.mode_used == gcb.MODE_COUNT
 
 
 def test_schedule_invariance_and_device_output():
@@ -203,6 +209,14 @@ def test_errors():
         gcb.Graph(3, torch.tensor([0, 1, 1, 1]), torch.tensor([1], dtype=torch.int32),
                   flags=gcb.VALIDATE)                                   # not symmetric
     assert e.value.code == -3
+    # an asymmetric adjacency SET (0 -> 1 only), not validated at create: the
+    # COUNT kernels detect it (underflow / stall) and report it, never a
+    # silently wrong colouring; Alg.4 has no fallback kernel
+    asym = gcb.Graph(3, torch.tensor([0, 1, 1, 1]), torch.tensor([1], dtype=torch.int32))
+    with pytest.raises(gcb.GCError) as e:
+        asym.color(1, gcb.JP_ALG4)
+    assert e.value.code == -3
+    asym.close()
     g = gcb.Graph(2, ro, torch.tensor([1, 0], dtype=torch.int32))
     with pytest.raises(gcb.GCError):
         g.color(1, gcb.MULTIHASH(17))
