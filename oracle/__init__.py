@@ -61,6 +61,8 @@ def lib():
         L.orc_color_luby.argtypes, L.orc_color_luby.restype = [i64, P, P, u64, P, P], i64
         L.orc_color_is_alg2.argtypes, L.orc_color_is_alg2.restype = [i64, P, P, u64, P, P], i64
         L.orc_color_jp_alg4.argtypes, L.orc_color_jp_alg4.restype = [i64, P, P, u64, P, P], i64
+        L.orc_color_hash_is.argtypes = [i64, P, P, u64, i32, P, P]
+        L.orc_color_hash_is.restype = i64
         L.orc_color_greedy.argtypes, L.orc_color_greedy.restype = [i64, P, P, P, P], i64
         L.orc_color_greedy_by_priority.argtypes = [i64, P, P, u64, P]
         L.orc_color_greedy_by_priority.restype = i64
@@ -170,6 +172,17 @@ def color_is_alg2(g, seed: int, with_stats: bool = False):
 def color_jp_alg4(g, seed: int, with_stats: bool = False):
     """GraphBLAS Jones-Plassmann, Alg.2 with Alg.4's frontier colour."""
     return _alg2(lib().orc_color_jp_alg4, g, seed, with_stats)
+
+
+def color_hash_is(g, seed: int, table: int, with_stats: bool = False):
+    """Hash IS colouring, Alg.6 made deterministic (R16-R20), table size T."""
+    n, ro, ci = _csr(g)
+    C = np.empty(max(n, 1), dtype=np.uint32)
+    rounds = np.zeros(1, dtype=np.int64)
+    r = lib().orc_color_hash_is(n, _pp(ro), _p(ci), seed, table, _pp(C), _pp(rounds))
+    if r < 0:
+        raise OracleError(f"orc_color_hash_is failed: {r}")
+    return (C[:n], int(r), int(rounds[0])) if with_stats else C[:n]
 
 
 def color_greedy(g, order=None):

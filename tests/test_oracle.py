@@ -15,6 +15,7 @@ import random
 
 import numpy as np
 import pytest
+import torch
 
 import graphgen as G
 import oracle as O
@@ -213,9 +214,70 @@ def test_golden_hand_derived(row):
         C = O.color_is_alg2(g, 1)
     elif variant == "jp_alg4":
         C = O.color_jp_alg4(g, 1)
+    elif variant.startswith("hash_is"):
+        C = O.color_hash_is(g, 1, int(variant[len("hash_is"):]))
     else:
         C = O.color_luby(g, 1)
     assert C.tolist() == expect
+
+
+# ------------------------------------------------ Hash IS, Alg.6
+@pytest.mark.parametrize("T", [0, 1, 3, 8])
+def test_hash_is_proper_complete_and_bounded(T):
+    for g in random_graphs(40, 60, seed0=700):
+        n = g.n
+        C, ncol, rounds = O.color_hash_is(g, 3, T, with_stats=True)
+        assert O.check_proper(g, C) == 0
+        assert (C != 0xFFFFFFFF).all()
+        assert ncol == np.unique(C).size
+        assert rounds <= 2 * n + 2  # R19: the heaviest uncoloured vertex wins within 2 rounds
+        assert C.max(initial=0) < 2 * max(rounds, 1)
+
+
+def test_hash_is_complete_graph_and_edgeless():
+    for n in (1, 2, 5, 9):
+        g = G.csr_from_lists(n, [(a, b) for a in range(n) for b in range(a + 1, n)])
+        C, ncol, rounds = O.color_hash_is(g, 7, n, with_stats=True)
+        # T >= Delta: every table holds both colours of each earlier round, so
+        # each round takes the heaviest and lightest remaining vertex with new
+        # colours: max-min's K_n closed form (n colours in ceil(n/2) rounds)
+        assert ncol == n and rounds == (n + 1) // 2
+        ref = O.color_maxmin(g, 7)
+        if n % 2:  # the lone vertex of the last round: max-min's R9 gives it the
+            ref[ref == n] = n - 1  # min colour 2k+1, Hash IS's R17 the max colour 2k
+        assert C.tolist() == ref.tolist()
+    g = G.csr_from_lists(6, [])
+    assert O.color_hash_is(g, 7, 0).tolist() == [0] * 6
+
+
+def test_hash_is_independent_of_row_order_and_duplicates():
+    # R16: the proposal is the heaviest / lightest of the set, not Alg.6's
+    # literal "last heavier neighbour", so entry order cannot matter
+    rng = np.random.default_rng(3)
+    for g in random_graphs(25, 80, seed0=900):
+        ro, ci = g.row_offsets.numpy(), g.col_indices.numpy().copy()
+        for v in range(g.n):
+            seg = ci[ro[v]:ro[v + 1]].copy()
+            rng.shuffle(seg)
+            ci[ro[v]:ro[v + 1]] = seg
+        h = G.Graph(g.n, g.row_offsets, torch.from_numpy(ci))
+        for T in (0, 2):
+            assert O.color_hash_is(g, 5, T).tolist() == O.color_hash_is(h, 5, T).tolist()
+
+
+def test_hash_is_large_table_reuses_colours():
+    # With T >= Delta a table holds every coloured neighbour's colour, so a
+    # reused colour never clashes with an old neighbour: every vertex's colour
+    # is either new in its round or absent from its neighbourhood -- and on
+    # sparse random graphs the reuse must beat max-min's count.
+    better = 0
+    for g in random_graphs(30, 120, seed0=1100):
+        deg = np.diff(g.row_offsets.numpy())
+        T = int(deg.max(initial=0)) + 1
+        C = O.color_hash_is(g, 11, T)
+        assert O.check_proper(g, C) == 0
+        better += np.unique(C).size <= np.unique(O.color_maxmin(g, 11)).size
+    assert better >= 25
 
 
 # ------------------------------------------------ Alg.2 / Alg.4
