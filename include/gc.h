@@ -73,12 +73,22 @@ typedef enum gc_status {
  * GC_JP_ALG4: Alg.2 with Alg.4 (reading R15): the same
  *   frontiers, each frontier takes ONE colour, the smallest colour not used by
  *   any coloured neighbour of the frontier (GraphBLAS Jones-Plassmann).
- *   COUNT mode only; single GPU. */
+ *   COUNT mode only; single GPU.
+ * GC_HASH_IS(t): the paper's Hash IS (Alg.6) made
+ *   deterministic (R16-R20): per round every uncoloured vertex
+ *   proposes the heaviest and the lightest of itself and its uncoloured
+ *   neighbours; a proposed vertex reuses the smallest colour used so far that
+ *   is not in its prohibited table of t colours (0 <= t <= 64), else takes a
+ *   new colour (2k max / 2k+1 min); conflicts reset the lighter endpoint (or
+ *   the new vertex, against an older colour).  Own per-round kernels
+ *   (gc_stats.mode_used = GC_MODE_SWEEP, options.mode ignored); single GPU. */
 #define GC_MAXMIN 0
 #define GC_LUBY_MIS 1
 #define GC_MULTIHASH(h) (2 | ((h) << 8))
 #define GC_IS_ALG2 3
 #define GC_JP_ALG4 4
+#define GC_HASH_IS(t) (5 | ((t) << 8))
+#define GC_HASH_TABLE_MAX 64
 #define GC_VARIANT_KIND(v) ((v) & 0xFF)
 #define GC_VARIANT_HASHES(v) (((v) >> 8) & 0xFF)
 

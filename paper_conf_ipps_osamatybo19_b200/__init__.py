@@ -33,6 +33,14 @@ def MULTIHASH(h: int) -> int:
     return 2 | (h << 8)
 
 
+HASH_TABLE_MAX = 64
+
+
+def HASH_IS(t: int) -> int:
+    """The paper's Hash IS (Alg.6, deterministic readings R16-R20), table of t colours."""
+    return 5 | (t << 8)
+
+
 BORROW_DEVICE = 1 << 0
 VALIDATE = 1 << 1
 COMPACT = 1 << 2

@@ -523,6 +523,11 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
             set_error("gc_color_ex: multi-hash needs 1 <= h <= 16");
             return GC_ERR_INVALID_ARG;
         }
+    } else if (kind == GC_HASH_IS(0)) {
+        if (GC_VARIANT_HASHES(o->variant) > GC_HASH_TABLE_MAX) {
+            set_error("gc_color_ex: hash IS needs a table of 0..64 colours");
+            return GC_ERR_INVALID_ARG;
+        }
     } else if (kind != GC_MAXMIN && kind != GC_LUBY_MIS && kind != GC_IS_ALG2 && kind != GC_JP_ALG4) {
         set_error("gc_color_ex: unknown variant");
         return GC_ERR_INVALID_ARG;
@@ -576,10 +581,17 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     RunResult res;
     auto run_count_variant = [&]() {
         if (g->count_unsafe) return (int)GC_ERR_NOT_SYMMETRIC;
-        if (jpv >= 1) return run_count_jp(g, p, &res, jpv);
+        if (jpv >= 1) {
+            int rs = ensure_strict_rows(g);
+            if (rs) return rs;
+            return run_count_jp(g, p, &res, jpv);
+        }
         return run_count_maxmin(g, p, &res);
     };
-    if (mode == GC_MODE_COUNT)
+    if (kind == GC_HASH_IS(0)) {
+        mode = GC_MODE_SWEEP;  // its own per-round kernels (gc_hash.cu)
+        rc = run_hash_is(g, p, GC_VARIANT_HASHES(o->variant), &res);
+    } else if (mode == GC_MODE_COUNT)
         rc = run_count_variant();
     else if (luby)
         rc = run_luby(g, p, &res);
@@ -634,7 +646,7 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     cudaEventElapsedTime(&ms, e0, e1);
     cudaEventDestroy(e0);
     cudaEventDestroy(e1);
-    if (!luby && (o->flags & GC_COMPACT) == 0) {
+    if (!luby && kind != GC_HASH_IS(0) && (o->flags & GC_COMPACT) == 0) {
         // raw colours are < 2RH; they must fit int32 (GC_ERR_TOO_LARGE otherwise)
         if ((uint64_t)2 * (uint64_t)res.rounds * (uint64_t)H > 0x7FFFFFFFull) {
             set_error("colours exceed INT32_MAX; use GC_COMPACT");

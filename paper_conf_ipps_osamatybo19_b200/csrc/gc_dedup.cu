@@ -44,7 +44,46 @@ __global__ void k_new_offsets(const int64_t *__restrict__ ro, int64_t n, int64_t
     }
 }
 
+__global__ void k_rows_strict(const int64_t *__restrict__ ro, const uint32_t *__restrict__ ci,
+                              int64_t n, unsigned int *bad) {
+    for (int64_t v = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; v < n;
+         v += (int64_t)gridDim.x * blockDim.x) {
+        const int64_t e1 = ro[v + 1];
+        for (int64_t e = ro[v] + 1; e < e1; ++e)
+            if (ci[e] <= ci[e - 1]) {
+                *bad = 1u;
+                break;
+            }
+    }
+}
 }  // namespace
+
+// Rows strictly increasing (no duplicates, sorted) -- checked once per handle.
+// The JP kernels (Luby-MIS, Alg.2, Alg.4 in COUNT mode) need a duplicate-free
+// adjacency before they start: a duplicate entry would be counted twice and
+// JP has no safe asymmetry detection, so the handle switches to its
+// deduplicated copy first when a row is not strictly increasing.
+int ensure_strict_rows(gc_graph *g) {
+    if (g->deduped || g->rows_strict) return GC_OK;
+    unsigned int *bad = nullptr;
+    unsigned int h = 0;
+    GC_CUDA_TRY(dmalloc(&bad, 4));
+    cudaError_t e = cudaMemsetAsync(bad, 0, 4, g->stream);
+    if (e == cudaSuccess && g->n > 0) {
+        k_rows_strict<<<g->sm_count * 8, 256, 0, g->stream>>>(g->ro, g->ci, g->n, bad);
+        e = cudaGetLastError();
+    }
+    if (e == cudaSuccess) e = cudaMemcpyAsync(&h, bad, 4, cudaMemcpyDeviceToHost, g->stream);
+    if (e == cudaSuccess) e = cudaStreamSynchronize(g->stream);
+    dfree(bad);
+    if (e != cudaSuccess) return cuda_fail(e, "row order check");
+    if (!h) {
+        g->rows_strict = true;
+        return GC_OK;
+    }
+    g->deduped = true;
+    return dedup_csr(g);
+}
 
 int dedup_csr(gc_graph *g) {
     const int64_t n = g->n, m = g->nnz;

@@ -385,7 +385,7 @@ int gc_create_csr_loopback(int64_t n, int64_t nnz, const int64_t *row_offsets,
 int64_t gc_color_dist(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_stats *stats) {
     Dist &d = *g->dist;
     const int kind = GC_VARIANT_KIND(o->variant);
-    if (kind == GC_LUBY_MIS || kind == GC_IS_ALG2 || kind == GC_JP_ALG4) {
+    if (kind == GC_LUBY_MIS || kind == GC_IS_ALG2 || kind == GC_JP_ALG4 || kind == GC_HASH_IS(0)) {
         set_error("distributed colouring supports GC_MAXMIN and GC_MULTIHASH(h)");
         return GC_ERR_INVALID_ARG;
     }

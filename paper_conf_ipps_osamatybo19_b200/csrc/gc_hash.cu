@@ -1,0 +1,354 @@
+// gc_hash.cu -- the paper's Hash IS colouring (Alg.6, P:L478-505, P:L557-614;
+// SURVEY N2) made deterministic by readings R16-R20.
+//
+// Round k over the frontier F_k (vertices uncoloured at the round's start),
+// five launches, every test reading the round-start state:
+//   k_hash_propose  8-lane group per v: mx(v) / mn(v) = heaviest / lightest of
+//                   {v} u (adj(v) n U_k) (R16); atomicOr of a max / min bit
+//                   into prop[mx] / prop[mn] (OR: order-free, so deterministic)
+//   k_hash_tent     thread per w: a proposed w takes the smallest used colour
+//                   not in its prohibited table (Alg.6 L20-24, R17), else the
+//                   new colour 2k (max-proposed) / 2k+1 (min only); a vertex
+//                   flagged by an earlier old-colour conflict takes the new
+//                   colour directly (R19)
+//   k_hash_resolve  8-lane group per tentatively coloured w: reset if an old
+//                   neighbour has its colour (code 2, sets the R19 flag) or a
+//                   heavier uncoloured neighbour has the same tentative colour
+//                   (code 1) (R18)
+//   k_hash_commit   thread per w: survivors write C[w], their round and the
+//                   used-colour bit; the rest are appended to F_{k+1}
+//   k_hash_table    8-lane group per v in F_{k+1}: insert the colours of the
+//                   neighbours coloured in round k, ascending, distinct, until
+//                   the table holds T (R20)
+// Frontier sizes live in device memory, so rounds are enqueued in batches
+// and the host reads the size once per batch (empty rounds are no-ops).
+#include <algorithm>
+
+#include "gc_internal.cuh"
+
+namespace gc {
+namespace {
+
+constexpr int kGroup = 8;  // lanes per vertex in the row-scanning kernels
+constexpr int kThreads = 256;
+constexpr uint32_t kNone = 0xFFFFFFFFu;
+
+struct HashArgs {
+    const int64_t *ro;
+    const uint32_t *ci;
+    uint32_t *C;
+    uint32_t *prop;   // bit 0: proposed as a max, bit 1: as a min
+    uint32_t *tent;   // tentative colour or kNone
+    uint8_t *res;     // resolve code: 0 keep, 1 new-new collision, 2 old colour
+    uint8_t *fresh;   // R19: must take a new colour
+    uint32_t *rnd;    // round in which the vertex was coloured (kNone before)
+    uint32_t *tab;    // T prohibited colours per vertex
+    uint8_t *tlen;    // entries used
+    uint32_t *used;   // bitmask of colours used so far
+    unsigned long long *ctr;  // [0], [1]: frontier sizes; [2]: rounds run
+    uint32_t key;
+    int T;
+};
+
+__device__ __forceinline__ uint32_t prio(const HashArgs &a, uint32_t v) { return weight_mix(v ^ a.key); }
+
+// The lanes of one vertex's group (groups of a warp diverge independently).
+__device__ __forceinline__ unsigned group_mask() {
+    return ((1u << kGroup) - 1u) << ((threadIdx.x & 31) & ~(kGroup - 1));
+}
+
+__device__ __forceinline__ unsigned long long group_max(unsigned long long x) {
+    const unsigned m = group_mask();
+#pragma unroll
+    for (int o = kGroup / 2; o > 0; o >>= 1) {
+        unsigned long long y = __shfl_xor_sync(m, x, o, kGroup);
+        x = y > x ? y : x;
+    }
+    return x;
+}
+__device__ __forceinline__ unsigned long long group_min(unsigned long long x) {
+    const unsigned m = group_mask();
+#pragma unroll
+    for (int o = kGroup / 2; o > 0; o >>= 1) {
+        unsigned long long y = __shfl_xor_sync(m, x, o, kGroup);
+        x = y < x ? y : x;
+    }
+    return x;
+}
+
+__global__ void k_hash_init(HashArgs a, uint32_t *F, int64_t n) {
+    for (int64_t v = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; v < n;
+         v += (int64_t)gridDim.x * blockDim.x) {
+        a.C[v] = GC_UNC;
+        a.prop[v] = 0;
+        a.fresh[v] = 0;
+        a.rnd[v] = kNone;
+        a.tlen[v] = 0;
+        F[v] = (uint32_t)v;
+    }
+}
+
+// Alg.6 L8-18 with R16: the heaviest / lightest of {v} u (adj(v) n U_k).
+__global__ void k_hash_propose(HashArgs a, const uint32_t *__restrict__ F, int in) {
+    const unsigned long long N = a.ctr[in];
+    const int lane = threadIdx.x % kGroup;
+    const int64_t groups = (int64_t)gridDim.x * (blockDim.x / kGroup);
+    for (int64_t i = ((int64_t)blockIdx.x * blockDim.x + threadIdx.x) / kGroup; i < (int64_t)N;
+         i += groups) {
+        const uint32_t v = F[i];
+        const unsigned long long self = ((unsigned long long)prio(a, v) << 32) | v;
+        unsigned long long mx = self, mn = self;
+        const int64_t e1 = a.ro[v + 1];
+        for (int64_t e = a.ro[v] + lane; e < e1; e += kGroup) {
+            const uint32_t u = a.ci[e];
+            if (a.C[u] != GC_UNC) continue;
+            const unsigned long long key = ((unsigned long long)prio(a, u) << 32) | u;
+            mx = key > mx ? key : mx;
+            mn = key < mn ? key : mn;
+        }
+        mx = group_max(mx);
+        mn = group_min(mn);
+        if (lane == 0) {
+            atomicOr(&a.prop[(uint32_t)mx], 1u);
+            atomicOr(&a.prop[(uint32_t)mn], 2u);
+        }
+    }
+}
+
+// Alg.6 L19-28 with R17 / R19.
+__global__ void k_hash_tent(HashArgs a, const uint32_t *__restrict__ F, int in, uint32_t k) {
+    const unsigned long long N = a.ctr[in];
+    for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < (int64_t)N;
+         i += (int64_t)gridDim.x * blockDim.x) {
+        const uint32_t w = F[i];
+        const uint32_t pr = a.prop[w];
+        uint32_t t = kNone;
+        if (pr) {
+            a.prop[w] = 0;  // ready for the next round
+            if (!a.fresh[w]) {
+                const uint32_t *tw = a.tab + (size_t)w * a.T;
+                const int len = a.tlen[w];
+                const uint32_t words = (2 * k + 31) / 32;  // used colours are < 2k
+                for (uint32_t wd = 0; wd < words && t == kNone; ++wd) {
+                    uint32_t bits = a.used[wd];
+                    while (bits) {
+                        const uint32_t c = wd * 32 + (uint32_t)__ffs(bits) - 1;
+                        bits &= bits - 1;
+                        bool in_tab = false;
+                        for (int j = 0; j < len; ++j) in_tab |= tw[j] == c;
+                        if (!in_tab) {
+                            t = c;
+                            break;
+                        }
+                    }
+                }
+            }
+            if (t == kNone) t = 2 * k + ((pr & 1u) ? 0u : 1u);
+        }
+        a.tent[w] = t;
+    }
+}
+
+// P:L501-505 with R18 / R19.
+__global__ void k_hash_resolve(HashArgs a, const uint32_t *__restrict__ F, int in) {
+    const unsigned long long N = a.ctr[in];
+    const int lane = threadIdx.x % kGroup;
+    const int64_t groups = (int64_t)gridDim.x * (blockDim.x / kGroup);
+    for (int64_t i = ((int64_t)blockIdx.x * blockDim.x + threadIdx.x) / kGroup; i < (int64_t)N;
+         i += groups) {
+        const uint32_t w = F[i];
+        const uint32_t t = a.tent[w];
+        if (t == kNone) continue;  // uniform over the group
+        const uint32_t pw = prio(a, w);
+        uint32_t code = 0;
+        const int64_t e1 = a.ro[w + 1];
+        for (int64_t e = a.ro[w] + lane; e < e1; e += kGroup) {
+            const uint32_t u = a.ci[e];
+            const uint32_t cu = a.C[u];
+            if (cu != GC_UNC) {
+                if (cu == t) code = 2;
+            } else if (a.tent[u] == t && prio(a, u) > pw) {
+                code = code > 1 ? code : 1;
+            }
+        }
+        code = (uint32_t)group_max(code);
+        if (lane == 0) a.res[w] = (uint8_t)code;
+    }
+}
+
+__global__ void k_hash_commit(HashArgs a, const uint32_t *__restrict__ F, int in, uint32_t *Fout,
+                              uint32_t k) {
+    const unsigned long long N = a.ctr[in];
+    if (blockIdx.x == 0 && threadIdx.x == 0 && N > 0) a.ctr[2] += 1;
+    const int64_t stride = (int64_t)gridDim.x * blockDim.x;
+    for (int64_t i0 = (int64_t)blockIdx.x * blockDim.x; i0 < (int64_t)N; i0 += stride) {
+        const int64_t i = i0 + threadIdx.x;
+        bool keep_unc = false;
+        if (i < (int64_t)N) {
+            const uint32_t w = F[i];
+            const uint32_t t = a.tent[w];
+            keep_unc = true;
+            if (t != kNone) {
+                const uint8_t r = a.res[w];
+                if (r == 0) {
+                    a.C[w] = t;
+                    a.rnd[w] = k;
+                    atomicOr(&a.used[t >> 5], 1u << (t & 31));
+                    keep_unc = false;
+                } else if (r == 2) {
+                    a.fresh[w] = 1;
+                }
+            }
+            if (keep_unc) {
+                // warp-aggregated append (frontier order does not matter:
+                // every decision of a round is a function of sets)
+                const unsigned mask = __activemask();
+                const unsigned bal = __ballot_sync(mask, 1);
+                const int leader = __ffs(bal) - 1;
+                const int lane = threadIdx.x & 31;
+                unsigned long long base = 0;
+                if (lane == leader) base = atomicAdd(&a.ctr[in ^ 1], (unsigned long long)__popc(bal));
+                base = __shfl_sync(mask, base, leader);
+                Fout[base + __popc(bal & ((1u << lane) - 1))] = w;
+            }
+        }
+    }
+}
+
+// P:L569-578 with R20: ascending insertion of the new neighbour colours.
+__global__ void k_hash_table(HashArgs a, const uint32_t *__restrict__ F, int in, uint32_t k) {
+    const unsigned long long N = a.ctr[in];
+    const int lane = threadIdx.x % kGroup;
+    const int64_t groups = (int64_t)gridDim.x * (blockDim.x / kGroup);
+    for (int64_t i = ((int64_t)blockIdx.x * blockDim.x + threadIdx.x) / kGroup; i < (int64_t)N;
+         i += groups) {
+        const uint32_t v = F[i];
+        int len = a.tlen[v];
+        if (len >= a.T) continue;
+        uint32_t *tv = a.tab + (size_t)v * a.T;
+        const int64_t e0 = a.ro[v], e1 = a.ro[v + 1];
+        long long last = -1;
+        while (len < a.T) {
+            // the smallest colour > last among the neighbours coloured in round k
+            unsigned long long best = ~0ull;
+            for (int64_t e = e0 + lane; e < e1; e += kGroup) {
+                const uint32_t u = a.ci[e];
+                if (a.rnd[u] != k) continue;
+                const unsigned long long c = a.C[u];
+                if ((long long)c > last && c < best) best = c;
+            }
+            best = group_min(best);
+            if (best == ~0ull) break;
+            last = (long long)best;
+            bool in_tab = false;
+            for (int j = 0; j < len; ++j) in_tab |= tv[j] == (uint32_t)best;
+            if (!in_tab) {
+                if (lane == 0) tv[len] = (uint32_t)best;
+                ++len;
+            }
+        }
+        if (lane == 0) a.tlen[v] = (uint8_t)len;
+    }
+}
+
+}  // namespace
+
+int run_hash_is(gc_graph *g, const RunParams &p, int T, RunResult *r) {
+    Scratch &s = g->s;
+    const int64_t n = g->n;
+    r->rounds = r->inner = r->launches = 0;
+    if (n == 0) return GC_OK;
+    if (n >= (1ll << 29)) {
+        set_error("hash IS: colours 2k with k <= 2n + 2 must fit int32 (n < 2^29)");
+        return GC_ERR_TOO_LARGE;
+    }
+    const size_t nn = (size_t)n;
+    const size_t used_words = (4 * nn + 64) / 32 + 1;
+    HashArgs a;
+    a.ro = g->ro;
+    a.ci = g->ci;
+    a.C = s.C;
+    a.key = p.keys.k[0];
+    a.T = T;
+    a.prop = a.tent = a.rnd = a.tab = a.used = nullptr;
+    a.res = a.fresh = a.tlen = nullptr;
+    a.ctr = nullptr;
+    int rc = GC_OK;
+    cudaStream_t st = g->stream;
+    const int grid = g->sm_count * 8;
+    const int64_t max_rounds = 2 * n + 4;
+    int64_t k = 0;
+    int cur = 0;
+    int batch = 4;
+    if (cudaSuccess != dmalloc(&a.prop, nn * 4) || cudaSuccess != dmalloc(&a.tent, nn * 4) ||
+        cudaSuccess != dmalloc(&a.rnd, nn * 4) || cudaSuccess != dmalloc(&a.res, nn) ||
+        cudaSuccess != dmalloc(&a.fresh, nn) || cudaSuccess != dmalloc(&a.tlen, nn) ||
+        cudaSuccess != dmalloc(&a.tab, nn * (size_t)std::max(T, 1) * 4) ||
+        cudaSuccess != dmalloc(&a.used, used_words * 4) || cudaSuccess != dmalloc(&a.ctr, 4 * 8)) {
+        rc = GC_ERR_OOM;
+        set_error("hash IS: device allocation failed");
+        goto out;
+    }
+    {
+        cudaError_t e = cudaMemsetAsync(a.used, 0, used_words * 4, st);
+        unsigned long long init[4] = {(unsigned long long)n, 0, 0, 0};
+        if (e == cudaSuccess) e = cudaMemcpyAsync(a.ctr, init, sizeof(init), cudaMemcpyHostToDevice, st);
+        if (e == cudaSuccess) {
+            k_hash_init<<<grid, kThreads, 0, st>>>(a, s.F[0], n);
+            e = cudaGetLastError();
+        }
+        if (e == cudaSuccess) e = cudaStreamSynchronize(st);  // `init` is a stack buffer
+        if (e != cudaSuccess) {
+            rc = cuda_fail(e, "hash IS init");
+            goto out;
+        }
+        r->launches += 1;
+        for (;;) {
+            for (int b = 0; b < batch; ++b, ++k) {
+                const int in = cur;
+                uint32_t *Fin = s.F[in], *Fout = s.F[in ^ 1];
+                e = cudaMemsetAsync(a.ctr + (in ^ 1), 0, 8, st);
+                if (e != cudaSuccess) break;
+                k_hash_propose<<<grid, kThreads, 0, st>>>(a, Fin, in);
+                k_hash_tent<<<grid, kThreads, 0, st>>>(a, Fin, in, (uint32_t)k);
+                k_hash_resolve<<<grid, kThreads, 0, st>>>(a, Fin, in);
+                k_hash_commit<<<grid, kThreads, 0, st>>>(a, Fin, in, Fout, (uint32_t)k);
+                if (T > 0) k_hash_table<<<grid, kThreads, 0, st>>>(a, Fout, in ^ 1, (uint32_t)k);
+                r->launches += T > 0 ? 5 : 4;
+                cur ^= 1;
+                e = cudaGetLastError();
+                if (e != cudaSuccess) break;
+            }
+            if (e == cudaSuccess)
+                e = cudaMemcpyAsync(s.host_pinned, a.ctr, 3 * 8, cudaMemcpyDeviceToHost, st);
+            if (e == cudaSuccess) e = cudaStreamSynchronize(st);
+            if (e != cudaSuccess) {
+                rc = cuda_fail(e, "hash IS rounds");
+                goto out;
+            }
+            const unsigned long long left = (unsigned long long)s.host_pinned[cur];
+            r->rounds = s.host_pinned[2];
+            if (left == 0) break;
+            if (k > max_rounds) {
+                set_error("hash IS: round bound 2n + 4 passed (asymmetric adjacency?)");
+                rc = GC_ERR_NOT_SYMMETRIC;
+                goto out;
+            }
+            batch = std::min(batch * 2, 64);
+        }
+    }
+    r->inner = r->rounds;
+out:
+    dfree(a.prop);
+    dfree(a.tent);
+    dfree(a.rnd);
+    dfree(a.res);
+    dfree(a.fresh);
+    dfree(a.tlen);
+    dfree(a.tab);
+    dfree(a.used);
+    dfree(a.ctr);
+    return rc;
+}
+
+}  // namespace gc

@@ -101,6 +101,7 @@ struct gc_graph {
     int sm_count = 148;
     bool count_unsafe = false;  // COUNT mode saw an asymmetric adjacency SET: use EVENT / SWEEP
     bool deduped = false;       // ro / ci were replaced by their deduplicated copy (gc_dedup.cu)
+    bool rows_strict = false;   // every row strictly increasing (checked once, gc_dedup.cu)
 };
 
 namespace gc {
@@ -201,8 +202,10 @@ int run_event_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int run_persistent_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int run_count_maxmin(gc_graph *g, const RunParams &p, RunResult *r);
 int dedup_csr(gc_graph *g);  // gc_dedup.cu
+int ensure_strict_rows(gc_graph *g);  // gc_dedup.cu: dedup first if a row is not strictly increasing
 int run_count_jp(gc_graph *g, const RunParams &p, RunResult *r, int jpv);  // 1 Luby, 2 Alg.2, 3 Alg.4
 int run_luby(gc_graph *g, const RunParams &p, RunResult *r);
+int run_hash_is(gc_graph *g, const RunParams &p, int T, RunResult *r);  // gc_hash.cu (Alg.6)
 int64_t count_colors_device(gc_graph *g, const uint32_t *C, int64_t n, bool compact,
                             uint32_t *C_inout, int64_t *launches);
 int launch_priorities(uint64_t seed, int j, int64_t v_begin, int64_t count, uint32_t *out,

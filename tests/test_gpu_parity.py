@@ -31,11 +31,15 @@ def _built():
 
 
 def variant_of(name: str, H: int = 1) -> int:
+    if name.startswith("hash_is"):
+        return gcb.HASH_IS(int(name[len("hash_is"):]))
     return {"maxmin": gcb.MAXMIN, "luby": gcb.LUBY_MIS, "is_alg2": gcb.IS_ALG2,
             "jp_alg4": gcb.JP_ALG4}.get(name, gcb.MULTIHASH(H))
 
 
 def oracle_colors(g, seed, variant, H=1):
+    if variant.startswith("hash_is"):
+        return O.color_hash_is(g, seed, int(variant[len("hash_is"):]))
     if variant == "luby":
         return O.color_luby(g, seed)
     if variant == "is_alg2":
@@ -53,6 +57,8 @@ def gpu_colors(g, seed, vcode, device_out=False, **kw):
 
 
 def supported_modes(vname, H):
+    if vname.startswith("hash_is"):
+        return [gcb.MODE_AUTO]  # its own per-round kernels; the mode is ignored
     if vname in ("is_alg2", "jp_alg4"):
         return [gcb.MODE_COUNT]
     return [gcb.MODE_SWEEP, gcb.MODE_COUNT] if vname == "luby" else MODES
@@ -122,6 +128,48 @@ def test_random_small_graphs(vname, H):
             assert k == (O.count_colors(ref) if n else 0)
 
 
+# ------------------------------------------- Hash IS, Alg.6
+@pytest.mark.parametrize("T", [0, 1, 4, 16, 64])
+def test_hash_is_random_small_graphs(T):
+    rng = random.Random(31 + T)
+    for i in range(80):
+        n = rng.randint(0, 400)
+        p = rng.choice([0.0, 0.01, 0.05, 0.2, 0.6])
+        g = G.random_graph(n, p, seed=7000 + 100 * T + i)
+        seed = rng.getrandbits(64)
+        ref, ncol, rounds = O.color_hash_is(g, seed, T, with_stats=True) if n else (
+            np.zeros(0, np.uint32), 0, 0)
+        C, k, st = gpu_colors(g, seed, gcb.HASH_IS(T))
+        assert (C == ref).all(), (i, n, p, T)
+        assert k == ncol and st.rounds == rounds
+
+
+@pytest.mark.parametrize("T", [0, 8])
+def test_hash_is_workload_graphs(T):
+    # several tiles and ragged tails: R-MAT (hubs, isolated vertices), ER, mesh, rgg
+    for g in (G.rmat(14, 16, seed=2), G.erdos_renyi(1 << 15, 8 << 15, seed=2), G.mesh3d(33, 31, 29),
+              G.rgg(13, seed=2)):
+        ref, ncol, rounds = O.color_hash_is(g, 1, T, with_stats=True)
+        C, k, st = gpu_colors(g, 1, gcb.HASH_IS(T), device_out=True)
+        assert (C == ref).all(), (g.name, T)
+        assert k == ncol and st.rounds == rounds
+        assert O.check_proper(g, C) == 0
+
+
+def test_hash_is_edge_cases():
+    cases = [G.csr_from_lists(1, []), G.csr_from_lists(33, []),
+             _csr_tensors(20001, [(0, i) for i in range(1, 20001)]),        # hub star
+             G.csr_from_lists(300, [(a, b) for a in range(300) for b in range(a + 1, 300)])]
+    for g in cases:
+        for T in (0, 2, 64):
+            ref = O.color_hash_is(g, 11, T)
+            C, k, _ = gpu_colors(g, 11, gcb.HASH_IS(T))
+            assert (C == ref).all(), (g.name, T)
+    with gcb.Graph(4, torch.tensor([0, 1, 2, 3, 3]), torch.tensor([1, 0, 3], dtype=torch.int32)) as h:
+        with pytest.raises(gcb.GCError):
+            h.color(1, gcb.HASH_IS(65), torch.empty(4, dtype=torch.int32))
+
+
 # --------------------------------------------------------------- edge cases
 def _csr_tensors(n, pairs):
     return G.csr_from_pairs(n, torch.tensor([a for a, _ in pairs], dtype=torch.int64),
@@ -183,6 +231,8 @@ def test_duplicates_and_unsorted_rows():
         C, _, st = gpu_colors(g2, 9, variant_of(vname))
         assert (C == oracle_colors(g, 9, vname)).all(), vname
         assert st.mode_used == gcb.MODE_COUNT
+    C, _, _ = gpu_colors(g2, 9, gcb.HASH_IS(3))
+    assert (C == O.color_hash_is(g, 9, 3)).all()
     C, _, st = gpu_colors(g2, 9, gcb.MULTIHASH(3), mode=gcb.MODE_COUNT)
     assert (C == O.color_maxmin(g, 9, 3)).all() and st.mode_used == gcb.MODE_COUNT
 
