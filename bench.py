@@ -42,8 +42,9 @@ def parse():
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--impl", default="gc", choices=["gc", "reference"])
     ap.add_argument("--scale", type=int, default=0, help="R-MAT scale (default 24+log2 N)")
-    ap.add_argument("--variant", default="maxmin", choices=["maxmin", "luby", "multihash"])
+    ap.add_argument("--variant", default="maxmin", choices=["maxmin", "luby", "multihash", "hash"])
     ap.add_argument("--hashes", type=int, default=4)
+    ap.add_argument("--table", type=int, default=8, help="Hash IS prohibited-table size T")
     ap.add_argument("--mode", default="auto", choices=["auto", "sweep", "event", "event-multi", "count"])
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-cpu-baseline", action="store_true")
@@ -143,7 +144,7 @@ def ncu_traffic(workload: str, kernel: str):
 
 
 # --------------------------------------------------------------- reference
-def cpu_sample(scale: int, variant: str, hashes: int):
+def cpu_sample(scale: int, variant: str, hashes: int, table: int = 8):
     """The oracle as it stands, on a bounded sample of the workload: a full
     colouring of the same generator at a smaller scale.  Returns dict."""
     import graphgen as G
@@ -153,6 +154,8 @@ def cpu_sample(scale: int, variant: str, hashes: int):
     t0 = time.perf_counter()
     if variant == "luby":
         O.color_luby(g, 1)
+    elif variant == "hash":
+        O.color_hash_is(g, 1, table)
     else:
         O.color_maxmin(g, 1, hashes if variant == "multihash" else 1)
     dt = time.perf_counter() - t0
@@ -175,6 +178,8 @@ def run_reference(args, rank, world):
         t0 = time.perf_counter()
         if args.variant == "luby":
             O.color_luby(g, 1)
+        elif args.variant == "hash":
+            O.color_hash_is(g, 1, args.table)
         else:
             O.color_maxmin(g, 1, args.hashes if args.variant == "multihash" else 1)
         dt = time.perf_counter() - t0
@@ -217,7 +222,8 @@ def main():
         dist.init_process_group("nccl", device_id=dev)
     scale = args.scale or (24 + int(round(math.log2(max(1, world)))))
     variant = {"maxmin": gcb.MAXMIN, "luby": gcb.LUBY_MIS,
-               "multihash": gcb.MULTIHASH(args.hashes)}[args.variant]
+               "multihash": gcb.MULTIHASH(args.hashes),
+               "hash": gcb.HASH_IS(args.table)}[args.variant]
     mode = {"auto": gcb.MODE_AUTO, "sweep": gcb.MODE_SWEEP, "event": gcb.MODE_EVENT,
             "event-multi": gcb.MODE_EVENT_MULTI, "count": gcb.MODE_COUNT}[args.mode]
 
@@ -295,6 +301,9 @@ def main():
                  gcb.MODE_SWEEP: {0: "k_sweep", 1: "k_hub", 2: "other", 3: "other"},
                  gcb.MODE_COUNT: {0: "k_count_persistent", 1: "k_count + k_count_hub",
                                   2: "init phase (round 0)", 3: "rounds"}}[sp.mode_used]
+        if args.variant == "hash":
+            names = {0: "k_hash_propose", 1: "k_hash_resolve", 2: "k_hash_table",
+                     3: "k_hash_tent + k_hash_commit"}
         if use_dist:
             names = {0: "k_dc_* round loop (COUNT, host-driven rounds + NCCL all-gathers)"
                      if sp.mode_used == gcb.MODE_COUNT else "sweep round loop",
@@ -375,7 +384,8 @@ def main():
 
     cpu = None
     if rank == 0 and world == 1 and not args.no_cpu_baseline:
-        cpu = cpu_sample(args.cpu_scale, args.variant, args.hashes)
+        cpu = cpu_sample(args.cpu_scale - (2 if args.variant == "hash" else 0), args.variant,
+                         args.hashes, args.table)
 
     if rank == 0:
         line = {"metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world,
@@ -384,6 +394,7 @@ def main():
                 "dtype": "u32", "data": "synthetic",
                 "config": {"workload": f"rmat-s{scale}-ef16 {args.variant}"
                                        + (f" H={args.hashes}" if args.variant == "multihash" else "")
+                                       + (f" T={args.table}" if args.variant == "hash" else "")
                                        + (" (cfg4)" if scale == 24 else
                                           " (cfg5)" if scale == 27 else ""),
                            "generator": "Graph500 Kronecker A,B,C=.57,.19,.19, symmetrised, "

@@ -32,6 +32,8 @@ namespace {
 constexpr int kGroup = 8;  // lanes per vertex in the row-scanning kernels
 constexpr int kThreads = 256;
 constexpr uint32_t kNone = 0xFFFFFFFFu;
+constexpr int64_t kLongMin = 512;  // rows longer than this go to a CTA (the *_long kernels)
+constexpr int kLongThreads = 512;
 
 struct HashArgs {
     const int64_t *ro;
@@ -45,7 +47,11 @@ struct HashArgs {
     uint32_t *tab;    // T prohibited colours per vertex
     uint8_t *tlen;    // entries used
     uint32_t *used;   // bitmask of colours used so far
-    unsigned long long *ctr;  // [0], [1]: frontier sizes; [2]: rounds run
+    uint32_t *wmx;    // last computed mx(v) / mn(v): still exact while uncoloured,
+    uint32_t *wmn;    // since U only shrinks (the max of a subset that keeps it)
+    unsigned long long *ctr;  // [0], [1]: frontier sizes; [2]: rounds run; [3..8] PROF;
+                              // [10 + c]: long rows of class c this round
+    uint32_t *longl[3];       // long rows deferred by class c (0 propose, 1 resolve, 2 table)
     uint32_t key;
     int T;
 };
@@ -76,6 +82,31 @@ __device__ __forceinline__ unsigned long long group_min(unsigned long long x) {
     return x;
 }
 
+__device__ __forceinline__ void push_long(const HashArgs &a, int c, uint32_t v) {
+    const unsigned long long i = atomicAdd(&a.ctr[10 + c], 1ull);
+    a.longl[c][i] = v;
+}
+
+// Block-wide max / min of a 64-bit key, result in every thread.
+template <bool MAX>
+__device__ __forceinline__ unsigned long long block_reduce(unsigned long long x) {
+    __shared__ unsigned long long sm[kLongThreads / 32];
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) {
+        unsigned long long y = __shfl_xor_sync(0xFFFFFFFFu, x, o);
+        x = MAX ? (y > x ? y : x) : (y < x ? y : x);
+    }
+    __syncthreads();  // sm reused across calls
+    if ((threadIdx.x & 31) == 0) sm[threadIdx.x >> 5] = x;
+    __syncthreads();
+    x = sm[0];
+    for (int i = 1; i < (int)(blockDim.x >> 5); ++i) {
+        const unsigned long long y = sm[i];
+        x = MAX ? (y > x ? y : x) : (y < x ? y : x);
+    }
+    return x;
+}
+
 __global__ void k_hash_init(HashArgs a, uint32_t *F, int64_t n) {
     for (int64_t v = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; v < n;
          v += (int64_t)gridDim.x * blockDim.x) {
@@ -84,11 +115,24 @@ __global__ void k_hash_init(HashArgs a, uint32_t *F, int64_t n) {
         a.fresh[v] = 0;
         a.rnd[v] = kNone;
         a.tlen[v] = 0;
+        a.wmx[v] = kNone;
+        a.wmn[v] = kNone;
         F[v] = (uint32_t)v;
     }
 }
 
 // Alg.6 L8-18 with R16: the heaviest / lightest of {v} u (adj(v) n U_k).
+// PROF: ctr[3 + 2c] += row entries scanned, ctr[4 + 2c] += rows scanned by
+// row-scan class c (0 propose, 1 resolve, 2 table).
+template <bool PROF>
+__device__ __forceinline__ void prof_row(const HashArgs &a, int c, int lane, int64_t len) {
+    if (PROF && lane == 0) {
+        atomicAdd(&a.ctr[3 + 2 * c], (unsigned long long)len);
+        atomicAdd(&a.ctr[4 + 2 * c], 1ull);
+    }
+}
+
+template <bool PROF>
 __global__ void k_hash_propose(HashArgs a, const uint32_t *__restrict__ F, int in) {
     const unsigned long long N = a.ctr[in];
     const int lane = threadIdx.x % kGroup;
@@ -96,21 +140,40 @@ __global__ void k_hash_propose(HashArgs a, const uint32_t *__restrict__ F, int i
     for (int64_t i = ((int64_t)blockIdx.x * blockDim.x + threadIdx.x) / kGroup; i < (int64_t)N;
          i += groups) {
         const uint32_t v = F[i];
+        {
+            // U_k is a subset of U_{k-1}: a cached argmax / argmin that is
+            // still uncoloured is still the argmax / argmin (no rescan)
+            const uint32_t cm = a.wmx[v], cn = a.wmn[v];
+            if (cm != kNone && a.C[cm] == GC_UNC && a.C[cn] == GC_UNC) {
+                if (lane == 0) {
+                    atomicOr(&a.prop[cm], 1u);
+                    atomicOr(&a.prop[cn], 2u);
+                }
+                continue;
+            }
+        }
+        const int64_t e0 = a.ro[v], e1 = a.ro[v + 1];
+        if (e1 - e0 > kLongMin) {
+            if (lane == 0) push_long(a, 0, v);
+            continue;
+        }
         const unsigned long long self = ((unsigned long long)prio(a, v) << 32) | v;
         unsigned long long mx = self, mn = self;
-        const int64_t e1 = a.ro[v + 1];
-        for (int64_t e = a.ro[v] + lane; e < e1; e += kGroup) {
+        for (int64_t e = e0 + lane; e < e1; e += kGroup) {
             const uint32_t u = a.ci[e];
             if (a.C[u] != GC_UNC) continue;
             const unsigned long long key = ((unsigned long long)prio(a, u) << 32) | u;
             mx = key > mx ? key : mx;
             mn = key < mn ? key : mn;
         }
+        prof_row<PROF>(a, 0, lane, e1 - e0);
         mx = group_max(mx);
         mn = group_min(mn);
         if (lane == 0) {
             atomicOr(&a.prop[(uint32_t)mx], 1u);
             atomicOr(&a.prop[(uint32_t)mn], 2u);
+            a.wmx[v] = (uint32_t)mx;
+            a.wmn[v] = (uint32_t)mn;
         }
     }
 }
@@ -150,7 +213,8 @@ __global__ void k_hash_tent(HashArgs a, const uint32_t *__restrict__ F, int in, 
 }
 
 // P:L501-505 with R18 / R19.
-__global__ void k_hash_resolve(HashArgs a, const uint32_t *__restrict__ F, int in) {
+template <bool PROF>
+__global__ void k_hash_resolve(HashArgs a, const uint32_t *__restrict__ F, int in, uint32_t k) {
     const unsigned long long N = a.ctr[in];
     const int lane = threadIdx.x % kGroup;
     const int64_t groups = (int64_t)gridDim.x * (blockDim.x / kGroup);
@@ -159,18 +223,33 @@ __global__ void k_hash_resolve(HashArgs a, const uint32_t *__restrict__ F, int i
         const uint32_t w = F[i];
         const uint32_t t = a.tent[w];
         if (t == kNone) continue;  // uniform over the group
-        const uint32_t pw = prio(a, w);
-        uint32_t code = 0;
-        const int64_t e1 = a.ro[w + 1];
-        for (int64_t e = a.ro[w] + lane; e < e1; e += kGroup) {
-            const uint32_t u = a.ci[e];
-            const uint32_t cu = a.C[u];
-            if (cu != GC_UNC) {
-                if (cu == t) code = 2;
-            } else if (a.tent[u] == t && prio(a, u) > pw) {
-                code = code > 1 ? code : 1;
-            }
+        const int64_t e0 = a.ro[w], e1 = a.ro[w + 1];
+        if (e1 - e0 > kLongMin) {
+            if (lane == 0) push_long(a, 1, w);
+            continue;
         }
+        const uint32_t pw = prio(a, w);
+        // an old neighbour can hold t only if t is not new (t < 2k) and the
+        // table may have missed colours (it is full); otherwise the first
+        // heavier collision decides (code 1), else the first old clash (2)
+        const uint32_t stop = (t < 2 * k && a.tlen[w] >= a.T) ? 2u : 1u;
+        const unsigned gm = group_mask();
+        uint32_t code = 0;
+        int64_t b = e0;
+        for (; b < e1; b += kGroup) {
+            const int64_t e = b + lane;
+            if (e < e1) {
+                const uint32_t u = a.ci[e];
+                const uint32_t cu = a.C[u];
+                if (cu != GC_UNC) {
+                    if (cu == t) code = 2;
+                } else if (a.tent[u] == t && prio(a, u) > pw) {
+                    code = code > 1 ? code : 1;
+                }
+            }
+            if (__any_sync(gm, code >= stop)) break;
+        }
+        prof_row<PROF>(a, 1, lane, (b + kGroup < e1 ? b + kGroup : e1) - e0);
         code = (uint32_t)group_max(code);
         if (lane == 0) a.res[w] = (uint8_t)code;
     }
@@ -216,6 +295,7 @@ __global__ void k_hash_commit(HashArgs a, const uint32_t *__restrict__ F, int in
 }
 
 // P:L569-578 with R20: ascending insertion of the new neighbour colours.
+template <bool PROF>
 __global__ void k_hash_table(HashArgs a, const uint32_t *__restrict__ F, int in, uint32_t k) {
     const unsigned long long N = a.ctr[in];
     const int lane = threadIdx.x % kGroup;
@@ -227,6 +307,10 @@ __global__ void k_hash_table(HashArgs a, const uint32_t *__restrict__ F, int in,
         if (len >= a.T) continue;
         uint32_t *tv = a.tab + (size_t)v * a.T;
         const int64_t e0 = a.ro[v], e1 = a.ro[v + 1];
+        if (e1 - e0 > kLongMin) {
+            if (lane == 0) push_long(a, 2, v);
+            continue;
+        }
         long long last = -1;
         while (len < a.T) {
             // the smallest colour > last among the neighbours coloured in round k
@@ -237,6 +321,7 @@ __global__ void k_hash_table(HashArgs a, const uint32_t *__restrict__ F, int in,
                 const unsigned long long c = a.C[u];
                 if ((long long)c > last && c < best) best = c;
             }
+            prof_row<PROF>(a, 2, lane, e1 - e0);
             best = group_min(best);
             if (best == ~0ull) break;
             last = (long long)best;
@@ -248,6 +333,97 @@ __global__ void k_hash_table(HashArgs a, const uint32_t *__restrict__ F, int in,
             }
         }
         if (lane == 0) a.tlen[v] = (uint8_t)len;
+    }
+}
+
+// The rows deferred by the group kernels, one CTA per row (hubs of R-MAT).
+template <bool PROF>
+__global__ void __launch_bounds__(kLongThreads) k_hash_propose_long(HashArgs a) {
+    const unsigned long long M = a.ctr[10];
+    for (unsigned long long it = blockIdx.x; it < M; it += gridDim.x) {
+        const uint32_t v = a.longl[0][it];
+        const int64_t e0 = a.ro[v], e1 = a.ro[v + 1];
+        const unsigned long long self = ((unsigned long long)prio(a, v) << 32) | v;
+        unsigned long long mx = self, mn = self;
+        for (int64_t e = e0 + threadIdx.x; e < e1; e += blockDim.x) {
+            const uint32_t u = a.ci[e];
+            if (a.C[u] != GC_UNC) continue;
+            const unsigned long long key = ((unsigned long long)prio(a, u) << 32) | u;
+            mx = key > mx ? key : mx;
+            mn = key < mn ? key : mn;
+        }
+        prof_row<PROF>(a, 0, threadIdx.x, e1 - e0);
+        mx = block_reduce<true>(mx);
+        mn = block_reduce<false>(mn);
+        if (threadIdx.x == 0) {
+            atomicOr(&a.prop[(uint32_t)mx], 1u);
+            atomicOr(&a.prop[(uint32_t)mn], 2u);
+            a.wmx[v] = (uint32_t)mx;
+            a.wmn[v] = (uint32_t)mn;
+        }
+    }
+}
+
+template <bool PROF>
+__global__ void __launch_bounds__(kLongThreads) k_hash_resolve_long(HashArgs a, uint32_t k) {
+    const unsigned long long M = a.ctr[11];
+    for (unsigned long long it = blockIdx.x; it < M; it += gridDim.x) {
+        const uint32_t w = a.longl[1][it];
+        const uint32_t t = a.tent[w];
+        const uint32_t pw = prio(a, w);
+        const int64_t e0 = a.ro[w], e1 = a.ro[w + 1];
+        const uint32_t stop = (t < 2 * k && a.tlen[w] >= a.T) ? 2u : 1u;  // as k_hash_resolve
+        unsigned long long code = 0;
+        int64_t b = e0;
+        for (; b < e1; b += blockDim.x) {
+            const int64_t e = b + threadIdx.x;
+            if (e < e1) {
+                const uint32_t u = a.ci[e];
+                const uint32_t cu = a.C[u];
+                if (cu != GC_UNC) {
+                    if (cu == t) code = 2;
+                } else if (a.tent[u] == t && prio(a, u) > pw) {
+                    code = code > 1 ? code : 1;
+                }
+            }
+            if (__syncthreads_or(code >= stop)) break;
+        }
+        prof_row<PROF>(a, 1, threadIdx.x, (b + (int64_t)blockDim.x < e1 ? b + blockDim.x : e1) - e0);
+        code = block_reduce<true>(code);
+        if (threadIdx.x == 0) a.res[w] = (uint8_t)code;
+    }
+}
+
+template <bool PROF>
+__global__ void __launch_bounds__(kLongThreads) k_hash_table_long(HashArgs a, uint32_t k) {
+    const unsigned long long M = a.ctr[12];
+    for (unsigned long long it = blockIdx.x; it < M; it += gridDim.x) {
+        const uint32_t v = a.longl[2][it];
+        int len = a.tlen[v];
+        uint32_t *tv = a.tab + (size_t)v * a.T;
+        const int64_t e0 = a.ro[v], e1 = a.ro[v + 1];
+        long long last = -1;
+        while (len < a.T) {  // uniform over the block
+            unsigned long long best = ~0ull;
+            for (int64_t e = e0 + threadIdx.x; e < e1; e += blockDim.x) {
+                const uint32_t u = a.ci[e];
+                if (a.rnd[u] != k) continue;
+                const unsigned long long c = a.C[u];
+                if ((long long)c > last && c < best) best = c;
+            }
+            prof_row<PROF>(a, 2, threadIdx.x, e1 - e0);
+            best = block_reduce<false>(best);
+            if (best == ~0ull) break;
+            last = (long long)best;
+            bool in_tab = false;
+            for (int j = 0; j < len; ++j) in_tab |= tv[j] == (uint32_t)best;
+            if (!in_tab) {
+                __syncthreads();  // every thread has read tv[0..len) before it grows
+                if (threadIdx.x == 0) tv[len] = (uint32_t)best;
+                ++len;
+            }
+        }
+        if (threadIdx.x == 0) a.tlen[v] = (uint8_t)len;
     }
 }
 
@@ -273,6 +449,9 @@ int run_hash_is(gc_graph *g, const RunParams &p, int T, RunResult *r) {
     a.prop = a.tent = a.rnd = a.tab = a.used = nullptr;
     a.res = a.fresh = a.tlen = nullptr;
     a.ctr = nullptr;
+    a.longl[0] = a.longl[1] = a.longl[2] = nullptr;
+    a.wmx = a.wmn = nullptr;
+    const size_t long_cap = (size_t)(g->nnz / kLongMin) + 1;
     int rc = GC_OK;
     cudaStream_t st = g->stream;
     const int grid = g->sm_count * 8;
@@ -280,18 +459,26 @@ int run_hash_is(gc_graph *g, const RunParams &p, int T, RunResult *r) {
     int64_t k = 0;
     int cur = 0;
     int batch = 4;
+    const bool has_long = g->max_deg > kLongMin;
+    const int grid_long = g->sm_count * 2;
+    const bool prof = p.prof && p.prof->on;
+    EventTimer tm;
     if (cudaSuccess != dmalloc(&a.prop, nn * 4) || cudaSuccess != dmalloc(&a.tent, nn * 4) ||
         cudaSuccess != dmalloc(&a.rnd, nn * 4) || cudaSuccess != dmalloc(&a.res, nn) ||
         cudaSuccess != dmalloc(&a.fresh, nn) || cudaSuccess != dmalloc(&a.tlen, nn) ||
         cudaSuccess != dmalloc(&a.tab, nn * (size_t)std::max(T, 1) * 4) ||
-        cudaSuccess != dmalloc(&a.used, used_words * 4) || cudaSuccess != dmalloc(&a.ctr, 4 * 8)) {
+        cudaSuccess != dmalloc(&a.used, used_words * 4) || cudaSuccess != dmalloc(&a.ctr, 16 * 8) ||
+        cudaSuccess != dmalloc(&a.wmx, nn * 4) || cudaSuccess != dmalloc(&a.wmn, nn * 4) ||
+        cudaSuccess != dmalloc(&a.longl[0], long_cap * 4) ||
+        cudaSuccess != dmalloc(&a.longl[1], long_cap * 4) ||
+        cudaSuccess != dmalloc(&a.longl[2], long_cap * 4)) {
         rc = GC_ERR_OOM;
         set_error("hash IS: device allocation failed");
         goto out;
     }
     {
         cudaError_t e = cudaMemsetAsync(a.used, 0, used_words * 4, st);
-        unsigned long long init[4] = {(unsigned long long)n, 0, 0, 0};
+        unsigned long long init[16] = {(unsigned long long)n};
         if (e == cudaSuccess) e = cudaMemcpyAsync(a.ctr, init, sizeof(init), cudaMemcpyHostToDevice, st);
         if (e == cudaSuccess) {
             k_hash_init<<<grid, kThreads, 0, st>>>(a, s.F[0], n);
@@ -308,13 +495,44 @@ int run_hash_is(gc_graph *g, const RunParams &p, int T, RunResult *r) {
                 const int in = cur;
                 uint32_t *Fin = s.F[in], *Fout = s.F[in ^ 1];
                 e = cudaMemsetAsync(a.ctr + (in ^ 1), 0, 8, st);
+                if (e == cudaSuccess && has_long) e = cudaMemsetAsync(a.ctr + 10, 0, 3 * 8, st);
                 if (e != cudaSuccess) break;
-                k_hash_propose<<<grid, kThreads, 0, st>>>(a, Fin, in);
-                k_hash_tent<<<grid, kThreads, 0, st>>>(a, Fin, in, (uint32_t)k);
-                k_hash_resolve<<<grid, kThreads, 0, st>>>(a, Fin, in);
-                k_hash_commit<<<grid, kThreads, 0, st>>>(a, Fin, in, Fout, (uint32_t)k);
-                if (T > 0) k_hash_table<<<grid, kThreads, 0, st>>>(a, Fout, in ^ 1, (uint32_t)k);
-                r->launches += T > 0 ? 5 : 4;
+                if (prof) {
+                    tm.begin(st, 0);
+                    k_hash_propose<true><<<grid, kThreads, 0, st>>>(a, Fin, in);
+                    if (has_long) k_hash_propose_long<true><<<grid_long, kLongThreads, 0, st>>>(a);
+                    tm.end(st);
+                    tm.begin(st, 3);
+                    k_hash_tent<<<grid, kThreads, 0, st>>>(a, Fin, in, (uint32_t)k);
+                    tm.end(st);
+                    tm.begin(st, 1);
+                    k_hash_resolve<true><<<grid, kThreads, 0, st>>>(a, Fin, in, (uint32_t)k);
+                    if (has_long) k_hash_resolve_long<true><<<grid_long, kLongThreads, 0, st>>>(a, (uint32_t)k);
+                    tm.end(st);
+                    tm.begin(st, 3);
+                    k_hash_commit<<<grid, kThreads, 0, st>>>(a, Fin, in, Fout, (uint32_t)k);
+                    tm.end(st);
+                    if (T > 0) {
+                        tm.begin(st, 2);
+                        k_hash_table<true><<<grid, kThreads, 0, st>>>(a, Fout, in ^ 1, (uint32_t)k);
+                        if (has_long)
+                            k_hash_table_long<true><<<grid_long, kLongThreads, 0, st>>>(a, (uint32_t)k);
+                        tm.end(st);
+                    }
+                } else {
+                    k_hash_propose<false><<<grid, kThreads, 0, st>>>(a, Fin, in);
+                    if (has_long) k_hash_propose_long<false><<<grid_long, kLongThreads, 0, st>>>(a);
+                    k_hash_tent<<<grid, kThreads, 0, st>>>(a, Fin, in, (uint32_t)k);
+                    k_hash_resolve<false><<<grid, kThreads, 0, st>>>(a, Fin, in, (uint32_t)k);
+                    if (has_long) k_hash_resolve_long<false><<<grid_long, kLongThreads, 0, st>>>(a, (uint32_t)k);
+                    k_hash_commit<<<grid, kThreads, 0, st>>>(a, Fin, in, Fout, (uint32_t)k);
+                    if (T > 0) {
+                        k_hash_table<false><<<grid, kThreads, 0, st>>>(a, Fout, in ^ 1, (uint32_t)k);
+                        if (has_long)
+                            k_hash_table_long<false><<<grid_long, kLongThreads, 0, st>>>(a, (uint32_t)k);
+                    }
+                }
+                r->launches += (T > 0 ? 5 : 4) + (has_long ? (T > 0 ? 3 : 2) : 0);
                 cur ^= 1;
                 e = cudaGetLastError();
                 if (e != cudaSuccess) break;
@@ -326,6 +544,7 @@ int run_hash_is(gc_graph *g, const RunParams &p, int T, RunResult *r) {
                 rc = cuda_fail(e, "hash IS rounds");
                 goto out;
             }
+            if (prof && (rc = tm.drain(p.prof))) goto out;
             const unsigned long long left = (unsigned long long)s.host_pinned[cur];
             r->rounds = s.host_pinned[2];
             if (left == 0) break;
@@ -338,6 +557,21 @@ int run_hash_is(gc_graph *g, const RunParams &p, int T, RunResult *r) {
         }
     }
     r->inner = r->rounds;
+    if (prof) {
+        // algorithmic bytes: a row scan reads the vertex id
+        // (4 B) and its offsets (16 B) and 4 B of col_indices per entry
+        // (status / weight gathers are L2-resident);
+        // tent + commit read / write 24 B per frontier vertex
+        unsigned long long c[16];
+        GC_CUDA_TRY(cudaMemcpy(c, a.ctr, sizeof(c), cudaMemcpyDeviceToHost));
+        int64_t frontier_sum = 0;
+        for (int cl = 0; cl < 3; ++cl) {
+            p.prof->bytes[cl] += 4 * (int64_t)c[3 + 2 * cl] + 20 * (int64_t)c[4 + 2 * cl];
+            p.prof->visits += (int64_t)c[3 + 2 * cl];
+        }
+        frontier_sum = (int64_t)c[4];  // propose scans every frontier row once
+        p.prof->bytes[3] += 24 * frontier_sum;
+    }
 out:
     dfree(a.prop);
     dfree(a.tent);
@@ -348,6 +582,9 @@ out:
     dfree(a.tab);
     dfree(a.used);
     dfree(a.ctr);
+    for (int c = 0; c < 3; ++c) dfree(a.longl[c]);
+    dfree(a.wmx);
+    dfree(a.wmn);
     return rc;
 }
 

@@ -159,7 +159,7 @@ def test_hash_is_workload_graphs(T):
 def test_hash_is_edge_cases():
     cases = [G.csr_from_lists(1, []), G.csr_from_lists(33, []),
              _csr_tensors(20001, [(0, i) for i in range(1, 20001)]),        # hub star
-             G.csr_from_lists(300, [(a, b) for a in range(300) for b in range(a + 1, 300)])]
+             G.csr_from_lists(700, [(a, b) for a in range(700) for b in range(a + 1, 700)])]  # CTA rows
     for g in cases:
         for T in (0, 2, 64):
             ref = O.color_hash_is(g, 11, T)

@@ -38,7 +38,21 @@ def run(name, g, variant, vname, mode="event", reps=5, warm=2, loopback=0):
     print(json.dumps(rec), flush=True)
 
 
+def main_hash():
+    """the Hash IS (Alg.6, deterministic) on every config, T = 0 / 8."""
+    dev = "cuda"
+    for cfg, name in (("cfg1", "cfg1 grid 64x64"), ("cfg2", "cfg2 ER 2^20 d16"),
+                      ("cfg3", "cfg3 mesh 128^3"), ("rgg", "N1 rgg_n_2_20"), ("cfg4", "cfg4 R-MAT s24")):
+        g = G.rgg(20, seed=1, device=dev) if cfg == "rgg" else G.config_graph(cfg, dev)
+        for T in (0, 8):
+            run(name, g, gcb.HASH_IS(T), f"hash IS T={T}", "auto")
+        run(name, g, gcb.MAXMIN, "maxmin", "auto")
+        del g
+
+
 def main():
+    if os.environ.get("GC_ONLY") == "hash":
+        return main_hash()
     dev = "cuda"
     g1 = G.config_graph("cfg1", dev)
     for m in ("count", "event", "sweep"):

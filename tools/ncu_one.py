@@ -13,8 +13,9 @@ ap.add_argument("--variant", default="maxmin")
 ap.add_argument("--warm", action="store_true")
 a = ap.parse_args()
 mode = {"event": gcb.MODE_EVENT, "sweep": gcb.MODE_SWEEP, "multi": gcb.MODE_EVENT_MULTI,
-        "count": gcb.MODE_COUNT}[a.mode]
-var = {"maxmin": gcb.MAXMIN, "luby": gcb.LUBY_MIS, "multihash": gcb.MULTIHASH(4)}[a.variant]
+        "count": gcb.MODE_COUNT, "auto": gcb.MODE_AUTO}[a.mode]
+var = {"maxmin": gcb.MAXMIN, "luby": gcb.LUBY_MIS, "multihash": gcb.MULTIHASH(4),
+       "hash": gcb.HASH_IS(8)}[a.variant]
 g = G.rmat(a.scale, 16, seed=1, device="cuda")
 torch.cuda.synchronize()
 out = torch.empty(g.n, dtype=torch.int32, device="cuda")
