@@ -259,10 +259,13 @@ __global__ void k_hash_commit(HashArgs a, const uint32_t *__restrict__ F, int in
                               uint32_t k) {
     const unsigned long long N = a.ctr[in];
     if (blockIdx.x == 0 && threadIdx.x == 0 && N > 0) a.ctr[2] += 1;
+    __shared__ unsigned s_cnt[kThreads / 32];
+    __shared__ unsigned long long s_base;
     const int64_t stride = (int64_t)gridDim.x * blockDim.x;
     for (int64_t i0 = (int64_t)blockIdx.x * blockDim.x; i0 < (int64_t)N; i0 += stride) {
         const int64_t i = i0 + threadIdx.x;
         bool keep_unc = false;
+        uint32_t wv = 0;
         if (i < (int64_t)N) {
             const uint32_t w = F[i];
             const uint32_t t = a.tent[w];
@@ -272,25 +275,36 @@ __global__ void k_hash_commit(HashArgs a, const uint32_t *__restrict__ F, int in
                 if (r == 0) {
                     a.C[w] = t;
                     a.rnd[w] = k;
-                    atomicOr(&a.used[t >> 5], 1u << (t & 31));
+                    // a set bit never clears: skip the (same-address) atomic when
+                    // it is already visible
+                    if (!(*(volatile uint32_t *)&a.used[t >> 5] & (1u << (t & 31))))
+                        atomicOr(&a.used[t >> 5], 1u << (t & 31));
                     keep_unc = false;
                 } else if (r == 2) {
                     a.fresh[w] = 1;
                 }
             }
-            if (keep_unc) {
-                // warp-aggregated append (frontier order does not matter:
-                // every decision of a round is a function of sets)
-                const unsigned mask = __activemask();
-                const unsigned bal = __ballot_sync(mask, 1);
-                const int leader = __ffs(bal) - 1;
-                const int lane = threadIdx.x & 31;
-                unsigned long long base = 0;
-                if (lane == leader) base = atomicAdd(&a.ctr[in ^ 1], (unsigned long long)__popc(bal));
-                base = __shfl_sync(mask, base, leader);
-                Fout[base + __popc(bal & ((1u << lane) - 1))] = w;
-            }
+            wv = w;
         }
+        // block-aggregated append, one global atomic per block and step
+        // (frontier order does not matter: every decision of a round is a
+        // function of sets)
+        const unsigned bal = __ballot_sync(0xFFFFFFFFu, keep_unc);
+        const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+        if (lane == 0) s_cnt[warp] = __popc(bal);
+        __syncthreads();
+        if (threadIdx.x == 0) {
+            unsigned tot = 0;
+            for (int j = 0; j < (int)(blockDim.x >> 5); ++j) {
+                const unsigned c = s_cnt[j];
+                s_cnt[j] = tot;
+                tot += c;
+            }
+            s_base = tot ? atomicAdd(&a.ctr[in ^ 1], (unsigned long long)tot) : 0ull;
+        }
+        __syncthreads();
+        if (keep_unc) Fout[s_base + s_cnt[warp] + __popc(bal & ((1u << lane) - 1))] = wv;
+        __syncthreads();  // s_cnt / s_base reused by the next step
     }
 }
 
