@@ -15,6 +15,8 @@ Parity status per function:
   color_is_alg2       pinned (golden, longest-decreasing-path DP, properness)
   color_jp_alg4       pinned (golden, K_n / edgeless closed forms, first-free
                       property per frontier, properness)
+  color_hash_is       pinned (golden at T = 0/1/4, K_n closed form, row-order
+                      invariance, properness, progress bound R <= 2n+2)
   paper-value parity  unpinned: the paper prints no colour count or worked
                       example for any variant (Fig.1b/3 unreadable).
 """
