@@ -34,6 +34,7 @@ constexpr int kThreads = 256;
 constexpr uint32_t kNone = 0xFFFFFFFFu;
 constexpr int64_t kLongMin = 512;  // rows longer than this go to a CTA (the *_long kernels)
 constexpr int kLongThreads = 512;
+constexpr int kTabOnePass = 8;  // table insertions done in one row pass (else repeated passes)
 
 struct HashArgs {
     const int64_t *ro;
@@ -323,6 +324,47 @@ __global__ void k_hash_table(HashArgs a, const uint32_t *__restrict__ F, int in,
         const int64_t e0 = a.ro[v], e1 = a.ro[v + 1];
         if (e1 - e0 > kLongMin) {
             if (lane == 0) push_long(a, 2, v);
+            continue;
+        }
+        if (a.T - len <= kTabOnePass) {
+            // one pass: every lane keeps its kTabOnePass smallest distinct new
+            // colours that are not in the table (sorted, padded with kNone);
+            // the group's smallest (T - len) are among their union
+            uint32_t buf[kTabOnePass];
+#pragma unroll
+            for (int j = 0; j < kTabOnePass; ++j) buf[j] = kNone;
+            for (int64_t e = e0 + lane; e < e1; e += kGroup) {
+                const uint32_t u = a.ci[e];
+                if (a.rnd[u] != k) continue;
+                const uint32_t c = a.C[u];
+                if (c >= buf[kTabOnePass - 1]) continue;
+                bool dup = false;
+#pragma unroll
+                for (int j = 0; j < kTabOnePass; ++j) dup |= buf[j] == c;
+                for (int j = 0; j < len; ++j) dup |= tv[j] == c;
+                if (dup) continue;
+                uint32_t cur = c;
+#pragma unroll
+                for (int j = 0; j < kTabOnePass; ++j) {  // sorted insert, drops the largest
+                    const uint32_t lo = min(buf[j], cur), hi = max(buf[j], cur);
+                    buf[j] = lo;
+                    cur = hi;
+                }
+            }
+            prof_row<PROF>(a, 2, lane, e1 - e0);
+            const int need = a.T - len;
+            for (int r = 0; r < need; ++r) {  // ascending merge of the lane lists
+                const uint32_t m = (uint32_t)group_min(buf[0]);
+                if (m == kNone) break;
+                if (lane == 0) tv[len] = m;
+                ++len;
+                if (buf[0] == m) {
+#pragma unroll
+                    for (int j = 0; j + 1 < kTabOnePass; ++j) buf[j] = buf[j + 1];
+                    buf[kTabOnePass - 1] = kNone;
+                }
+            }
+            if (lane == 0) a.tlen[v] = (uint8_t)len;
             continue;
         }
         long long last = -1;
