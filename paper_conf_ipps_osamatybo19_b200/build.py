@@ -38,23 +38,51 @@ def needs_build() -> bool:
     return any(os.path.getmtime(p) > t for p in deps)
 
 
-def build(force: bool = False, verbose: bool = False) -> str:
-    if not force and not needs_build():
-        return OUT
+OBJ = os.path.join(ROOT, "build", "obj")
+
+
+def build(force: bool = False, verbose: bool = False, out: str = OUT, defines=()) -> str:
+    """One object per .cu (compiled in parallel, rebuilt when the source or a
+    header is newer), then one nvcc link step into `out`."""
+    if not force and out == OUT and not defines and not needs_build():
+        return out
+    from concurrent.futures import ThreadPoolExecutor
+
     inc, libd = nccl_dirs()
-    cmd = [NVCC, "-gencode", "arch=compute_100a,code=sm_100a", "-O3", "-lineinfo", "-std=c++17",
-           "-Xcompiler", "-fPIC", "-shared", "-I" + os.path.join(ROOT, "include")]
+    flags = [NVCC, "-gencode", "arch=compute_100a,code=sm_100a", "-O3", "-lineinfo", "-std=c++17",
+             "-Xcompiler", "-fPIC", "-I" + os.path.join(ROOT, "include")]
+    flags += ["-D" + d for d in defines]
     if inc:
-        cmd += ["-DGC_HAVE_NCCL=1", "-I" + inc, "-L" + libd, "-Xlinker", "-rpath=" + libd,
-                "-l:libnccl.so.2"]
+        flags += ["-DGC_HAVE_NCCL=1", "-I" + inc]
     if verbose:
-        cmd += ["-Xptxas", "-v"]
-    tmp = OUT + f".tmp{os.getpid()}"
-    cmd += ["-o", tmp] + sources()
-    subprocess.check_call(cmd)
-    os.replace(tmp, OUT)
-    return OUT
+        flags += ["-Xptxas", "-v"]
+    tag = "_".join(d.replace("=", "") for d in defines) or "default"
+    odir = os.path.join(OBJ, tag)
+    os.makedirs(odir, exist_ok=True)
+    hdrs = glob.glob(os.path.join(CSRC, "*.cuh")) + [os.path.join(ROOT, "include", "gc.h")]
+    t_hdr = max(os.path.getmtime(h) for h in hdrs)
+
+    def one(src):
+        obj = os.path.join(odir, os.path.basename(src) + ".o")
+        if force or not os.path.exists(obj) or os.path.getmtime(obj) < max(os.path.getmtime(src), t_hdr):
+            tmpo = obj + f".tmp{os.getpid()}"
+            subprocess.check_call(flags + ["-c", "-o", tmpo, src])
+            os.replace(tmpo, obj)
+        return obj
+
+    with ThreadPoolExecutor(max_workers=min(8, os.cpu_count() or 1)) as ex:
+        objs = list(ex.map(one, sources()))
+    link = [NVCC, "-gencode", "arch=compute_100a,code=sm_100a", "-shared", "-Xcompiler", "-fPIC"]
+    if inc:
+        link += ["-L" + libd, "-Xlinker", "-rpath=" + libd, "-l:libnccl.so.2"]
+    tmp = out + f".tmp{os.getpid()}"
+    subprocess.check_call(link + ["-o", tmp] + objs)
+    os.replace(tmp, out)
+    return out
 
 
 if __name__ == "__main__":
-    print(build(force="--force" in sys.argv, verbose="-v" in sys.argv))
+    # python -m paper_conf_ipps_osamatybo19_b200.build [--force] [-v] [-DNAME=V ... --out PATH]
+    defs = [a[2:] for a in sys.argv[1:] if a.startswith("-D")]
+    o = sys.argv[sys.argv.index("--out") + 1] if "--out" in sys.argv else OUT
+    print(build(force="--force" in sys.argv, verbose="-v" in sys.argv, out=o, defines=defs))

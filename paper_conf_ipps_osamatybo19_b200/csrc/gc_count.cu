@@ -60,6 +60,11 @@
 #endif
 constexpr bool kCountStream = GC_COUNT_STREAM != 0;
 
+#ifndef GC_PROF_UNIT
+#define GC_PROF_UNIT 0  // 1 (PROF builds only): per-round latency breakdown of the WL units
+                        // (item load, column ids, atomics) in round_stats slots 9, 11-15
+#endif
+
 #ifndef GC_PACKED
 #define GC_PACKED 0  // 1: 32-bit (hi << 16 | lo) round counts -- max-min only (no JP / multi-hash branch);
                      // measured 27.9 vs 28.1 ms on R-MAT s24, not worth the restriction
@@ -371,8 +376,10 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
     __syncthreads();
     if (prs && threadIdx.x == 0) {
         const unsigned long long fdt = gtimer() - st.t_fs;  // this block's fresh step
-        red_add(prs + 11, fdt);
-        red_max(prs + 12, fdt);
+        if (!GC_PROF_UNIT) {
+            red_add(prs + 11, fdt);
+            red_max(prs + 12, fdt);
+        }
         red_add(prs + 2, (unsigned long long)st.vis);
         red_max(prs + 5, gtimer() - t_round);
         st.vis = 0;
@@ -490,12 +497,18 @@ template <int Q, bool JP = false, bool WIDE = false>
 __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, int64_t e,
                                      int64_t end, int stride, uint32_t k, uint32_t &nvis,
                                      unsigned long long *mask = nullptr, uint32_t *sbits = nullptr,
-                                     bool want_mex = false, bool want_set = false) {
+                                     bool want_mex = false, bool want_set = false,
+                                     long long *tprof = nullptr) {
     uint32_t w[Q];
 #pragma unroll
     for (int q = 0; q < Q; ++q) {
         const int64_t eq = e + (int64_t)q * stride;
         w[q] = (v != kNone && eq < end) ? __ldcs(a.ci + eq) : kNone;
+    }
+    if (GC_PROF_UNIT && tprof) {
+#pragma unroll
+        for (int q = 0; q < Q; ++q) asm volatile("" ::"r"(w[q]));
+        tprof[0] = clock64();
     }
     if (!JP && GC_SKIP_COLOURED) {  // coloured neighbours: no atomic (their counts are dead)
         uint32_t mb[Q];
@@ -561,6 +574,11 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
                 }
             }
         }
+    }
+    if (GC_PROF_UNIT && tprof) {
+#pragma unroll
+        for (int q = 0; q < Q; ++q) asm volatile("" ::"l"((unsigned long long)old[q]));
+        tprof[1] = clock64();
     }
     bool fresh[Q];
 #pragma unroll
@@ -780,8 +798,8 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
     if (prs && threadIdx.x == 0) {  // PROF: this block's units are done
         const unsigned long long dt = gtimer() - t_round;
         red_max(prs + 7, dt);
-        red_max(prs + 9, ~dt);  // min via ~
-        red_max(prs + 13, (unsigned long long)st.nf);
+        if (!GC_PROF_UNIT) red_max(prs + 9, ~dt);  // min via ~
+        if (!GC_PROF_UNIT) red_max(prs + 13, (unsigned long long)st.nf);
         st.t_fs = gtimer();
     }
     const unsigned nf = min(st.nf, (unsigned)kStF);
@@ -1139,11 +1157,30 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                 } else {
                     const bool cl = !JP && (it.lf & kFirst) && lane == 0;
                     const uint32_t z = cl ? __ldcg(a.Zlo + it.v) : 0u;
+                    long long tp[3] = {0, 0, 0};
+                    if (GC_PROF_UNIT && prs) {
+                        asm volatile("" ::"r"(pv));
+                        tp[2] = clock64();
+                    }
                     if (MH)
                         walk_mh<kSeg / 32>(a, it.v, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k, nvis);
                     else
-                        walk<kSeg / 32, JP>(a, it.v, pv, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k, nvis);
+                        walk<kSeg / 32, JP>(a, it.v, pv, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k, nvis,
+                                            nullptr, nullptr, false, false, (GC_PROF_UNIT && prs) ? tp : nullptr);
                     if (cl) colour_fin<MH>(a, it.v, it.lf, k, z);
+                    if (GC_PROF_UNIT && prs && !MH) {
+                        // max over the warp's lanes of each stage's end (cycles since the unit start)
+                        const unsigned mi = __reduce_max_sync(kFull, (unsigned)(tp[2] - c_unit));
+                        const unsigned mc = __reduce_max_sync(kFull, (unsigned)(tp[0] - c_unit));
+                        const unsigned ma = __reduce_max_sync(kFull, (unsigned)(tp[1] - c_unit));
+                        if (lane == 0) {
+                            red_max(prs + 12, mi);
+                            red_max(prs + 14, mc);
+                            red_max(prs + 15, ma);
+                            red_add(prs + 11, mc);        // sum: unit start -> column ids in
+                            red_add(prs + 9, ma - mc);    // sum: column ids -> atomics back
+                        }
+                    }
                 }
             } else if (lane_rows) {
                 // short rows: one per lane, 4 entries per step
@@ -1214,7 +1251,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                 }
             }
             if (prs && lane == 0)
-                red_max(prs + 10, (unsigned long long)(clock64() - c_unit));
+                red_max(prs + ((GC_PROF_UNIT && u >= nw) ? 13 : 10), (unsigned long long)(clock64() - c_unit));
         }
         sl0 = sl1;
         wl0 = wl1;

@@ -1,6 +1,6 @@
 """Per round: decrements per vertex (max / top), from a COUNT-mode colouring of R-MAT."""
 import sys, os, json
-sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.dirname(os.path.abspath(__file__)))))
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
 import torch
 import graphgen as G
 import paper_conf_ipps_osamatybo19_b200 as gcb
