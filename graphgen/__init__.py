@@ -221,15 +221,42 @@ def rmat_pairs(scale: int, edge_factor: int = 16, seed: int = 1, device="cpu",
         yield _label_permutation(u, scale, seed), _label_permutation(v, scale, seed)
 
 
-def rmat(scale: int, edge_factor: int = 16, seed: int = 1, device="cpu") -> Graph:
-    """R-MAT / Graph500 Kronecker graph, symmetrised (cfg4: s24, cfg5: s27)."""
+def rmat(scale: int, edge_factor: int = 16, seed: int = 1, device="cpu", pieces: int = 1) -> Graph:
+    """R-MAT / Graph500 Kronecker graph, symmetrised (cfg4: s24, cfg5: s27).
+
+    pieces > 1 builds the same CSR row range by row range (each range keeps
+    the pairs touching it from a fresh pass over the counter-based pair
+    stream), so peak memory is about 1/pieces of the one-shot build (cfg5)."""
     n = 1 << scale
-    us, vs = [], []
-    for u, v in rmat_pairs(scale, edge_factor, seed, device):
-        us.append(u); vs.append(v)
-    return csr_from_pairs(n, torch.cat(us), torch.cat(vs), f"rmat_s{scale}_ef{edge_factor}",
-                          {"kind": "rmat", "scale": scale, "edge_factor": edge_factor,
-                           "seed": seed})
+    meta = {"kind": "rmat", "scale": scale, "edge_factor": edge_factor, "seed": seed}
+    name = f"rmat_s{scale}_ef{edge_factor}"
+    if pieces <= 1:
+        us, vs = [], []
+        for u, v in rmat_pairs(scale, edge_factor, seed, device):
+            us.append(u); vs.append(v)
+        return csr_from_pairs(n, torch.cat(us), torch.cat(vs), name, meta)
+    step = (n + pieces - 1) // pieces
+    ros, cis, base = [], [], 0
+    for v0 in range(0, n, step):
+        v1 = min(n, v0 + step)
+        keys = []
+        for u, v in rmat_pairs(scale, edge_factor, seed, device):
+            keep = u != v
+            u, v = u[keep], v[keep]
+            for a, b in ((u, v), (v, u)):
+                m = (a >= v0) & (a < v1)
+                keys.append((a[m] - v0) * n + b[m])
+        k = torch.unique(torch.cat(keys), sorted=True)
+        del keys
+        rows = k // n
+        cis.append((k - rows * n).to(torch.int32))
+        del k
+        ro = torch.cumsum(torch.bincount(rows, minlength=v1 - v0), 0) + base
+        del rows
+        ros.append(ro)
+        base = int(ro[-1]) if ro.numel() else base
+    ro = torch.cat([torch.zeros(1, dtype=torch.int64, device=device)] + ros)
+    return Graph(n, ro, torch.cat(cis), name, meta)
 
 
 def rgg(scale: int, seed: int = 1, device="cpu", radius_coef: float = 0.55) -> Graph:

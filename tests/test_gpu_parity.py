@@ -8,6 +8,7 @@ every vertex, alongside the frontier-size trace of a smaller R-MAT.
 """
 from __future__ import annotations
 
+import os
 import random
 
 import numpy as np
@@ -478,6 +479,56 @@ def test_cfg5_style_partitioned_rmat_s25():
     C = one.cpu().numpy().view(np.uint32)
     gh = g.to("cpu")
     assert O.cert_maxmin(gh, 1, 1, C) == 0
+
+
+def test_cfg5_rmat_s27_one_gpu_and_partitions():
+    """cfg5 at its stated size: R-MAT s27 ef16 (1.3e8 vertices, nnz > 2^31).
+    One B200 colours it through gc_create_csr / AUTO (the bench launch
+    configuration); the partitioned algorithm (loopback transport: the same
+    COUNT rounds, ghost rows and pair exchange as over NCCL) at P = 2, 4, 8
+    equals P = 1 bit for bit; on the host the oracle's O(m)
+    certificate -- which determines the max-min colouring uniquely (App. C
+    #4, mutation-pinned in test_oracle.py) -- checks every vertex, plus
+    properness and n_colors in {2R-1, 2R}."""
+    g = G.rmat(27, 16, seed=1, device="cuda", pieces=8)
+    assert g.n == 1 << 27 and g.nnz > 2 ** 31
+    with gcb.Graph(g.n, g.row_offsets, g.col_indices, flags=gcb.BORROW_DEVICE) as h:
+        one = torch.empty(g.n, dtype=torch.int32, device="cuda")
+        _, k1, st1 = h.color(1, gcb.MAXMIN, one, stats=True)
+    assert st1.mode_used == gcb.MODE_COUNT
+    for parts in (2, 4, 8):
+        with gcb.loopback_graph(g.n, g.row_offsets, g.col_indices, parts) as h:
+            outp = torch.empty(g.n, dtype=torch.int32, device="cuda")
+            _, kp, stp = h.color(1, gcb.MAXMIN, outp, stats=True)
+        assert stp.mode_used == gcb.MODE_COUNT
+        assert torch.equal(outp, one) and kp == k1 and stp.rounds == st1.rounds, parts
+        del outp
+        gcb.trim()
+    C = one.cpu().numpy().view(np.uint32)
+    gh = g.to("cpu")
+    del g, one
+    torch.cuda.empty_cache()
+    assert O.cert_maxmin(gh, 1, 1, C) == 0
+    assert O.check_proper(gh, C) == 0
+    assert k1 == O.count_colors(C) and k1 in (2 * st1.rounds - 1, 2 * st1.rounds)
+
+
+@pytest.mark.skipif(os.environ.get("GC_SLOW_TESTS") != "1",
+                    reason="about 10 min of oracle time on the host: GC_SLOW_TESTS=1")
+def test_cfg4_rmat_s24_full_oracle_elementwise():
+    """The bench graph (R-MAT s24) against the full oracle colouring (Alg.1 +
+    Alg.5 with snapshot rounds, not the certificate), element by element,
+    with the round count and the per-round frontier sizes."""
+    g = G.config_graph("cfg4", device="cuda")
+    with gcb.Graph(g.n, g.row_offsets, g.col_indices, flags=gcb.BORROW_DEVICE) as h:
+        out = torch.empty(g.n, dtype=torch.int32, device="cuda")
+        _, k, st = h.color(1, gcb.MAXMIN, out, stats=True, frontier_cap=1 << 14)
+    C = out.cpu().numpy().view(np.uint32)
+    gh = g.to("cpu")
+    del g
+    ref, R, nk = O.color_maxmin(gh, 1, with_stats=True)
+    assert (C == ref).all()
+    assert st.rounds == R and st.frontier_sizes == nk and k == O.count_colors(ref)
 
 
 @pytest.mark.parametrize("vname", ["is_alg2", "jp_alg4"])

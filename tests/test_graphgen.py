@@ -55,3 +55,11 @@ def test_label_permutation_is_bijective():
     x = torch.arange(1 << 12)
     y = G._label_permutation(x, 12, seed=9)
     assert torch.equal(torch.sort(y).values, x)
+
+
+def test_rmat_built_by_pieces_is_identical():
+    """The range-by-range build (used for cfg5, s27) yields the same CSR."""
+    a = G.rmat(13, 16, seed=4)
+    for pieces in (2, 3, 8):
+        b = G.rmat(13, 16, seed=4, pieces=pieces)
+        assert torch.equal(a.row_offsets, b.row_offsets) and torch.equal(a.col_indices, b.col_indices)

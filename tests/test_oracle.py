@@ -399,6 +399,45 @@ def test_certificate_accepts_and_rejects():
                 assert O.cert_maxmin(g, 4, H, D) != 0
 
 
+def _first_improper(g, C):
+    """1 + the first vertex (ascending) that is uncoloured or shares its colour
+    with a neighbour, 0 if none: P:L40-44 written out with numpy."""
+    ro, ci = g.row_offsets.numpy(), g.col_indices.numpy().astype(np.int64)
+    src = np.repeat(np.arange(g.n), np.diff(ro))
+    bad = C == O.UNCOLORED
+    clash = C[src] == C[ci]
+    bad[src[clash]] = True
+    idx = np.flatnonzero(bad)
+    return int(idx[0]) + 1 if idx.size else 0
+
+
+def test_check_proper_rejects_mutations():
+    """orc_check_proper (the problem definition) is pinned by what it
+    must reject: on true colourings, recolouring one endpoint of a random edge
+    to the other's colour and uncolouring a random vertex are both reported,
+    at exactly the first offending vertex a numpy restatement finds; a
+    colouring proper by construction (all colours distinct) is accepted."""
+    rng = random.Random(31)
+    for g in random_graphs(30, 60, seed0=90):
+        C = O.color_maxmin(g, 5)
+        assert O.check_proper(g, C) == 0 == _first_improper(g, C)
+        assert O.check_proper(g, np.arange(g.n, dtype=np.uint32)) == 0
+        ro, ci = g.row_offsets.numpy(), g.col_indices.numpy()
+        for _ in range(10 if g.nnz else 0):
+            e = rng.randrange(g.nnz)
+            u = int(np.searchsorted(ro, e, side="right") - 1)
+            w = int(ci[e])
+            D = C.copy()
+            D[u] = D[w]
+            bad = O.check_proper(g, D)
+            assert bad != 0 and bad - 1 <= min(u, w) and bad == _first_improper(g, D)
+        v = rng.randrange(g.n)
+        D = C.copy()
+        D[v] = O.UNCOLORED
+        bad = O.check_proper(g, D)
+        assert bad != 0 and bad - 1 <= v and bad == _first_improper(g, D)
+
+
 def test_chromatic_lower_bound():
     for g in random_graphs(40, 8, seed0=31):
         adj = adjacency(g)
