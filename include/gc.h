@@ -47,7 +47,10 @@ typedef enum gc_status {
                                   col >= n, nnz mismatch, bad variant/options */
     GC_ERR_SELF_LOOP = -2,     /* a self-loop never terminates (Alg.5 L29-34
                                   with u = v fails both strict tests; R7) */
-    GC_ERR_NOT_SYMMETRIC = -3, /* only checked with GC_VALIDATE */
+    GC_ERR_NOT_SYMMETRIC = -3, /* gc_create_csr: with GC_VALIDATE; gc_color: Alg.2 / Alg.4 in COUNT
+                                  mode (and the partitioned COUNT rounds) when the adjacency SETS
+                                  are not symmetric (the other variants fall back to the witness /
+                                  sweep kernels instead) */
     GC_ERR_TOO_LARGE = -4,     /* n >= 2^32, or colours would pass INT32_MAX */
     GC_ERR_CUDA = -5,          /* CUDA runtime error / no usable device */
     GC_ERR_NCCL = -6,          /* NCCL error in the distributed path */
@@ -149,13 +152,14 @@ typedef struct gc_options {
 /* Statistics filled by gc_color_ex (optional). */
 typedef struct gc_stats {
     uint32_t struct_size;     /* sizeof(gc_stats) */
-    int32_t mode_used;        /* GC_MODE_SWEEP, GC_MODE_EVENT or GC_MODE_EVENT_MULTI */
+    int32_t mode_used;        /* GC_MODE_SWEEP, GC_MODE_EVENT, GC_MODE_EVENT_MULTI or GC_MODE_COUNT */
     int64_t rounds;           /* R: rounds (max-min / multi-hash) or colours (Luby) */
     int64_t inner_iterations; /* Luby: Alg.3 do-while iterations; else == rounds */
     int64_t n_colors;         /* distinct colours */
     int64_t launches;         /* kernels launched by this call */
     double ms;                /* device time of the call (CUDA events) */
-    int64_t *frontier_sizes;  /* optional caller buffer: N_k per round */
+    int64_t *frontier_sizes;  /* optional caller buffer: N_k per round (not written for
+                                 Luby-MIS and GC_HASH_IS) */
     int64_t frontier_cap;     /* its capacity */
     /* GC_PROFILE only.  Kernel classes: [0] the per-round sweep kernel (the
      * hot loop), [1] the hub (CTA-per-row) kernel, [2] everything else.

@@ -125,6 +125,17 @@ def _check(rc: int) -> int:
     return rc
 
 
+def _numel(t) -> int:
+    return int(t.numel()) if hasattr(t, "numel") else int(t.size)
+
+
+def _need(t, count: int, what: str) -> None:
+    """The C side reads / writes `count` elements of `t`: a shorter buffer
+    would be an out-of-bounds access, so it is rejected here."""
+    if t is not None and _numel(t) < count:
+        raise ValueError(f"{what}: {_numel(t)} elements, {count} needed")
+
+
 def _ptr(t, dtypes):
     """Pointer of a contiguous torch tensor or numpy array with an allowed dtype."""
     if t is None:
@@ -167,7 +178,10 @@ class Graph:
     def __init__(self, n: int, row_offsets, col_indices, flags: int = 0):
         self._h = ctypes.c_void_p()
         self.n = int(n)
-        self.nnz = int(col_indices.numel() if hasattr(col_indices, "numel") else col_indices.size)
+        self.nnz = _numel(col_indices)
+        self.out_len = self.n  # colours written by color() (dist handles: see dist_graph)
+        if self.n >= 0 and _numel(row_offsets) != self.n + 1:
+            raise ValueError(f"row_offsets: {_numel(row_offsets)} elements, n + 1 = {self.n + 1} needed")
         self._keep = (row_offsets, col_indices) if flags & BORROW_DEVICE else None
         _check(lib().gc_create_csr(self.n, self.nnz, _ptr(row_offsets, ("int64",)),
                                    _ptr(col_indices, ("int32", "uint32")), flags,
@@ -177,6 +191,7 @@ class Graph:
     def _from_handle(cls, h, n, nnz, keep=None):
         obj = cls.__new__(cls)
         obj._h, obj.n, obj.nnz, obj._keep = h, n, nnz, keep
+        obj.out_len = n
         return obj
 
     def set_stream(self, stream) -> None:
@@ -191,9 +206,11 @@ class Graph:
         """Colour the graph.  `out`: int32 tensor/array of n entries on host or
         device (allocated on the host if None).  Returns (out, n_colors) or
         (out, n_colors, ColorStats) with stats=True."""
+        need = self.local_len if (flags & OUT_LOCAL_SLICE and hasattr(self, "local_len")) else self.out_len
         if out is None:
             import torch
-            out = torch.empty(self.n, dtype=torch.int32)
+            out = torch.empty(need, dtype=torch.int32)
+        _need(out, need, "out")
         o = gc_options()
         o.struct_size = ctypes.sizeof(gc_options)
         o.variant, o.seed, o.flags, o.mode = variant, seed, flags, mode
@@ -243,7 +260,9 @@ class Graph:
 def loopback_graph(n: int, row_offsets, col_indices, parts: int, flags: int = 0) -> Graph:
     """The partitioned (multi-GPU) algorithm with `parts` partitions on this GPU."""
     h = ctypes.c_void_p()
-    nnz = int(col_indices.numel() if hasattr(col_indices, "numel") else col_indices.size)
+    nnz = _numel(col_indices)
+    if _numel(row_offsets) != n + 1:
+        raise ValueError(f"row_offsets: {_numel(row_offsets)} elements, n + 1 = {n + 1} needed")
     _check(lib().gc_create_csr_loopback(n, nnz, _ptr(row_offsets, ("int64",)),
                                         _ptr(col_indices, ("int32", "uint32")), parts, flags,
                                         ctypes.byref(h)))
@@ -260,7 +279,10 @@ def dist_graph(n_global: int, v_begin: int, v_end: int, row_offsets_local, col_i
                unique_id: bytes, rank: int, world: int, flags: int = 0) -> Graph:
     """A rank's share of a 1D-partitioned graph (collective over `world` ranks)."""
     h = ctypes.c_void_p()
-    nnz = int(col_indices_global.numel())
+    nnz = _numel(col_indices_global)
+    if _numel(row_offsets_local) != v_end - v_begin + 1:
+        raise ValueError(f"row_offsets_local: {_numel(row_offsets_local)} elements, "
+                         f"{v_end - v_begin + 1} needed")
     uid = ctypes.create_string_buffer(bytes(unique_id), 128)
     _check(lib().gc_create_csr_dist(n_global, v_begin, v_end, nnz,
                                     _ptr(row_offsets_local, ("int64",)),
@@ -269,6 +291,7 @@ def dist_graph(n_global: int, v_begin: int, v_end: int, row_offsets_local, col_i
     g = Graph._from_handle(h, n_global, nnz,
                            keep=(row_offsets_local, col_indices_global) if flags & BORROW_DEVICE
                            else None)
+    g.local_len = v_end - v_begin  # GC_OUT_LOCAL_SLICE writes the owned range only
     return g
 
 
@@ -280,6 +303,7 @@ def color(n, row_offsets, col_indices, seed=1, variant=MAXMIN, out=None, **kw):
 
 def priorities(seed: int, j: int, v_begin: int, count: int, out):
     """a0: out[i] = p_j(v_begin + i) computed on the GPU (host or device out)."""
+    _need(out, count, "out")
     _check(lib().gc_priorities(seed, j, v_begin, count, _ptr(out, ("int32", "uint32"))))
     return out
 

@@ -72,7 +72,8 @@ def build(force: bool = False, verbose: bool = False, out: str = OUT, defines=()
 
     with ThreadPoolExecutor(max_workers=min(8, os.cpu_count() or 1)) as ex:
         objs = list(ex.map(one, sources()))
-    link = [NVCC, "-gencode", "arch=compute_100a,code=sm_100a", "-shared", "-Xcompiler", "-fPIC"]
+    link = [NVCC, "-gencode", "arch=compute_100a,code=sm_100a", "-shared", "-Xcompiler", "-fPIC",
+            "-Xlinker", "--no-undefined"]
     if inc:
         link += ["-L" + libd, "-Xlinker", "-rpath=" + libd, "-l:libnccl.so.2"]
     tmp = out + f".tmp{os.getpid()}"

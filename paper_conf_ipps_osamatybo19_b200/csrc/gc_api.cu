@@ -574,10 +574,11 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     prof.on = (o->flags & GC_PROFILE) != 0;
     p.prof = &prof;
 
-    cudaEvent_t e0, e1;
-    GC_CUDA_TRY(cudaEventCreate(&e0));
-    GC_CUDA_TRY(cudaEventCreate(&e1));
-    GC_CUDA_TRY(cudaEventRecord(e0, g->stream));
+    EventPair ev;  // destroyed on every exit path
+    GC_CUDA_TRY(cudaEventCreate(&ev.e0));
+    GC_CUDA_TRY(cudaEventCreate(&ev.e1));
+    GC_CUDA_TRY(cudaEventRecord(ev.e0, g->stream));
+    cudaEvent_t e0 = ev.e0, e1 = ev.e1;
     RunResult res;
     auto run_count_variant = [&]() {
         if (g->count_unsafe) return (int)GC_ERR_NOT_SYMMETRIC;
@@ -605,9 +606,15 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
         // The counts need a symmetric adjacency MULTISET; duplicate entries are
         // legal input (adjacency sets decide the colouring).  Switch the handle
         // once to its deduplicated, row-sorted copy and rerun (gc_dedup.cu).
-        g->deduped = true;
-        rc = dedup_csr(g);
+        rc = dedup_csr(g);  // sets g->deduped on success only
         if (!rc) rc = run_count_variant();
+        else if (rc == GC_ERR_OOM || rc == GC_ERR_TOO_LARGE) rc = GC_ERR_NOT_SYMMETRIC;  // no copy: fall back
+    }
+    if (rc == GC_ERR_TOO_LARGE && mode == GC_MODE_COUNT && jpv < 2) {
+        // a round's item count overflowed the persistent kernel's round word
+        // (gc_count.cu, trap 9): the EVENT / SWEEP kernels have no such field
+        g->count_unsafe = true;
+        rc = GC_ERR_NOT_SYMMETRIC;
     }
     if (rc == GC_ERR_NOT_SYMMETRIC && mode == GC_MODE_COUNT && jpv < 2) {
         // Still asymmetric after deduplication: the adjacency SETS are not
@@ -627,11 +634,7 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
             if (!rc) rc = run_persistent_maxmin(g, p, &res);
         }
     }
-    if (rc) {
-        cudaEventDestroy(e0);
-        cudaEventDestroy(e1);
-        return rc;
-    }
+    if (rc) return rc;
     int64_t launches = res.launches;
     int64_t ncol = count_colors_device(g, g->s.C, g->n, (o->flags & GC_COMPACT) != 0, g->s.C,
                                        &launches);
@@ -644,8 +647,6 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     GC_CUDA_TRY(cudaEventSynchronize(e1));
     float ms = 0.f;
     cudaEventElapsedTime(&ms, e0, e1);
-    cudaEventDestroy(e0);
-    cudaEventDestroy(e1);
     if (!luby && kind != GC_HASH_IS(0) && (o->flags & GC_COMPACT) == 0) {
         // raw colours are < 2RH; they must fit int32 (GC_ERR_TOO_LARGE otherwise)
         if ((uint64_t)2 * (uint64_t)res.rounds * (uint64_t)H > 0x7FFFFFFFull) {
@@ -677,7 +678,8 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
                 GC_CUDA_TRY(cudaMemcpy(stats->round_stats, g->s.rstat, sizeof(int64_t) * 16 * m,
                                        cudaMemcpyDeviceToHost));
         }
-        if (stats->frontier_sizes && stats->frontier_cap > 0 && !luby) {
+        // (Hash IS keeps no per-round frontier trace: its entries are left untouched)
+        if (stats->frontier_sizes && stats->frontier_cap > 0 && !luby && kind != GC_HASH_IS(0)) {
             int64_t m = std::min<int64_t>(std::min<int64_t>(stats->frontier_cap, res.rounds),
                                           g->s.nk_cap);
             if (m > 0)

@@ -1695,6 +1695,10 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
     const bool mh = !jp && p.H > 1;
     r->rounds = r->inner = r->launches = 0;
     if (n == 0) return GC_OK;
+    if (n >= (1ll << 29)) {  // a round's SL items could pass the round word's 29-bit field
+        set_error("COUNT mode: n >= 2^29 exceeds the round word's item field");
+        return GC_ERR_TOO_LARGE;
+    }
     int rc = ensure_count_scratch(g);
     if (rc) return rc;
     if (mh && s.cnt_h < p.H) {  // H count words per vertex
@@ -1814,6 +1818,10 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
         else
             snprintf(buf, sizeof(buf), "internal consistency check %llu failed in round %llu (vertex %llu)",
                      h[cErr], h[cErr + 1], h[cErr + 2]);
+        if (h[cErr] == 9) {  // one round reserved more items than the round word's fields hold
+            set_error("COUNT mode: a round's items overflowed the round word (2^29 short / 2^24 long items)");
+            return GC_ERR_TOO_LARGE;
+        }
         set_error(buf);
         return (h[cErr] == 4 || h[cErr] == 5 || h[cErr] == 7) ? GC_ERR_NOT_SYMMETRIC : GC_ERR_CUDA;
     }

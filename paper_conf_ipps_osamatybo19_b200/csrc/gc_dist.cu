@@ -124,6 +124,34 @@ int exchange(gc_graph *g, size_t bytes, SendF send, RecvF recv) {
 
 }  // namespace
 
+// The handle's rows were replaced by their deduplicated copy (gc_dedup.cu):
+// point every partition at its rows of the new CSR and drop its COUNT state
+// (ghost rows and list capacities follow the rows).
+int dist_reslice(gc_graph *g) {
+    Dist &d = *g->dist;
+    if (!d.loopback) {
+        Part &p = d.parts[0];
+        p.ro = g->ro;
+        p.ci = g->ci;
+        p.nnz = g->nnz;
+        free_dist_count(p);
+        return GC_OK;
+    }
+    std::vector<int64_t> h_ro((size_t)d.n_global + 1);
+    GC_CUDA_TRY(cudaMemcpyAsync(h_ro.data(), g->ro, sizeof(int64_t) * h_ro.size(), cudaMemcpyDeviceToHost,
+                                g->stream));
+    GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
+    for (Part &p : d.parts) {
+        p.nnz = h_ro[p.v1] - h_ro[p.v0];
+        p.ci = g->ci + h_ro[p.v0];
+        k_rebase<<<64, 256, 0, g->stream>>>(g->ro + p.v0, p.v1 - p.v0, p.ro);
+        free_dist_count(p);
+    }
+    GC_CUDA_TRY(cudaGetLastError());
+    return GC_OK;
+}
+
+
 int dist_exchange(gc_graph *g, size_t bytes, const std::vector<const void *> &send,
                   const std::vector<void *> &recv) {
     return exchange(g, bytes, [&](int q) { return send[q]; }, [&](int q) { return recv[q]; });

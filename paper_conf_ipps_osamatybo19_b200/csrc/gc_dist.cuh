@@ -61,6 +61,7 @@ struct Dist {
 
 int run_dist_count(gc_graph *g, const RunParams &p, RunResult *r, int64_t *frontier, int64_t fcap);
 void free_dist_count(Part &p);
+int dist_reslice(gc_graph *g);  // after gc_dedup.cu replaced the handle's rows
 int dist_exchange(gc_graph *g, size_t bytes, const std::vector<const void *> &send,
                   const std::vector<void *> &recv);
 int nccl_fail(int e, const char *what);

@@ -431,6 +431,14 @@ int run_dist_count(gc_graph *g, const RunParams &p, RunResult *r, int64_t *front
     const uint32_t key = p.keys.k[0];
     r->rounds = r->inner = r->launches = 0;
     const int blocks = g->sm_count * 8;
+    if (!g->deduped && !g->rows_strict) {
+        // the counts need a symmetric adjacency MULTISET: duplicate entries
+        // (legal input, R13) are removed from this rank's rows first -- the
+        // same adjacency sets, so the same colouring on every rank
+        int rc = ensure_strict_rows(g);
+        if (rc) return rc;
+        if (g->deduped && (rc = dist_reslice(g))) return rc;
+    }
     for (auto &pt : d.parts) {
         int rc = ensure_dc(g, pt, n);
         if (rc) return rc;

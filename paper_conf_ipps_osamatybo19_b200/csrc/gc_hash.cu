@@ -629,6 +629,9 @@ int run_hash_is(gc_graph *g, const RunParams &p, int T, RunResult *r) {
         p.prof->bytes[3] += 24 * frontier_sum;
     }
 out:
+    // on an error path kernels may still be queued: the blocks go back to the
+    // cache only when no pending work uses them (gc_alloc.cu contract)
+    if (rc) cudaStreamSynchronize(st);
     dfree(a.prop);
     dfree(a.tent);
     dfree(a.rnd);

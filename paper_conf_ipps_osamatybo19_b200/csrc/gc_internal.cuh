@@ -106,6 +106,15 @@ struct gc_graph {
 
 namespace gc {
 
+// A pair of CUDA events destroyed with the scope (every exit path).
+struct EventPair {
+    cudaEvent_t e0 = nullptr, e1 = nullptr;
+    ~EventPair() {
+        if (e0) cudaEventDestroy(e0);
+        if (e1) cudaEventDestroy(e1);
+    }
+};
+
 // ----------------------------------------------------------------- errors
 void set_error(const std::string &msg);
 int cuda_fail(cudaError_t e, const char *what);

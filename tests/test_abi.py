@@ -51,10 +51,33 @@ def test_library_is_sm100a_only(libgc):
     assert "sm_100a" in out
 
 
-def test_struct_layouts_match_header(libgc):
-    # gc_options / gc_stats sizes as compiled in C (see include/gc.h)
-    assert ctypes.sizeof(gcb.gc_options) == 4 + 4 + 8 + 4 + 4 + 4 + 4 + 4 + 28
-    assert ctypes.sizeof(gcb.gc_stats) == 4 + 4 + 8 * 4 + 8 + 8 + 8 + 8 * 4 * 3 + 8 + 8 * 4
+def _compile_and_run(src: str) -> str:
+    import tempfile
+    with tempfile.TemporaryDirectory() as d:
+        c, exe = os.path.join(d, "t.c"), os.path.join(d, "t")
+        open(c, "w").write(src)
+        subprocess.check_call(["gcc", "-I" + os.path.join(ROOT, "include"), "-o", exe, c])
+        return subprocess.check_output([exe]).decode()
+
+
+def test_struct_layouts_match_header():
+    """sizeof / offsetof of every field of gc_options and gc_stats as the C
+    compiler lays out include/gc.h, against the binding's ctypes structures."""
+    lines = ['#include <stdio.h>', '#include <stddef.h>', '#include "gc.h"', 'int main(void){']
+    for st in (gcb.gc_options, gcb.gc_stats):
+        name = st.__name__
+        lines.append(f'printf("{name} size %zu\\n", sizeof({name}));')
+        for f, _ in st._fields_:
+            lines.append(f'printf("{name} {f} %zu\\n", offsetof({name}, {f}));')
+    lines.append("return 0;}")
+    got = {}
+    for ln in _compile_and_run("\n".join(lines) + "\n").splitlines():
+        st, f, v = ln.split()
+        got[(st, f)] = int(v)
+    for st in (gcb.gc_options, gcb.gc_stats):
+        assert got[(st.__name__, "size")] == ctypes.sizeof(st), st.__name__
+        for f, _ in st._fields_:
+            assert got[(st.__name__, f)] == getattr(st, f).offset, (st.__name__, f)
 
 
 def test_fails_loudly_without_gpu(libgc):
@@ -95,3 +118,28 @@ def test_variant_codes_match_header():
         got = [int(x) for x in subprocess.check_output([exe]).split()]
     assert got == [gcb.MAXMIN, gcb.LUBY_MIS, gcb.MULTIHASH(4), gcb.IS_ALG2, gcb.JP_ALG4,
                    gcb.HASH_IS(8), gcb.HASH_TABLE_MAX]
+
+
+def test_binding_rejects_short_buffers():
+    """The binding checks every buffer the C side reads or writes against the
+    sizes it passes: a short array raises ValueError before any
+    call reaches libgc -- no out-of-bounds device or host access."""
+    import numpy as np
+    import torch
+    ro = torch.tensor([0, 1, 2], dtype=torch.int64)
+    ci = torch.tensor([1, 0], dtype=torch.int32)
+    with pytest.raises(ValueError, match="row_offsets"):
+        gcb.Graph(3, ro, ci)  # n + 1 = 4 offsets needed
+    with pytest.raises(ValueError, match="row_offsets"):
+        gcb.loopback_graph(1, ro, ci, 2)
+    with pytest.raises(ValueError, match="out"):
+        gcb.priorities(1, 0, 0, 8, torch.empty(4, dtype=torch.int32))
+    with pytest.raises(ValueError, match="out"):
+        gcb.priorities(1, 0, 0, 8, np.empty(7, dtype=np.uint32))
+    g = gcb.Graph._from_handle(ctypes.c_void_p(), 10, 0)  # no device needed: rejected first
+    with pytest.raises(ValueError, match="out"):
+        g.color(1, gcb.MAXMIN, torch.empty(9, dtype=torch.int32))
+    g.local_len = 4  # a rank's owned range (dist_graph)
+    with pytest.raises(ValueError, match="out"):
+        g.color(1, gcb.MAXMIN, torch.empty(3, dtype=torch.int32), flags=gcb.OUT_LOCAL_SLICE)
+    g._h = ctypes.c_void_p()

@@ -236,6 +236,42 @@ def test_duplicates_and_unsorted_rows():
     assert (C == O.color_hash_is(g, 9, 3)).all()
     C, _, st = gpu_colors(g2, 9, gcb.MULTIHASH(3), mode=gcb.MODE_COUNT)
     assert (C == O.color_maxmin(g, 9, 3)).all() and st.mode_used == gcb.MODE_COUNT
+    # the partitioned COUNT rounds deduplicate each partition's rows first
+    # (one-sided duplicates would break the count multiset): same colouring
+    # at every P, in COUNT mode
+    for parts in (1, 2, 4):
+        with gcb.loopback_graph(g2.n, g2.row_offsets, g2.col_indices, parts) as h:
+            out = torch.empty(g2.n, dtype=torch.int32)
+            _, _, st = h.color(9, gcb.MAXMIN, out, stats=True)
+            assert st.mode_used == gcb.MODE_COUNT
+            assert (out.numpy().view(np.uint32) == ref).all(), parts
+
+
+def test_dedup_in_row_batches(monkeypatch):
+    """The deduplicated copy is built in row batches of < 2^30 entries (CUB's
+    int sizes; cfg5 has nnz > 2^31): a tiny batch size (test hook) forces many
+    batches, rows longer than a batch included; same colourings."""
+    monkeypatch.setenv("GC_DEDUP_BATCH", "700")
+    rng = random.Random(4)
+    g = G.rmat(12, 16, seed=8)
+    ref = O.color_maxmin(g, 2)
+    ro, ci = g.row_offsets.tolist(), g.col_indices.tolist()
+    rows = []
+    for v in range(g.n):
+        r = ci[ro[v]:ro[v + 1]]
+        r = r + rng.sample(r, min(len(r), 3))
+        rng.shuffle(r)
+        rows.append(r)
+    nro = [0]
+    for r in rows:
+        nro.append(nro[-1] + len(r))
+    assert max(len(r) for r in rows) > 700
+    g2 = G.Graph(g.n, torch.tensor(nro, dtype=torch.int64),
+                 torch.tensor([x for r in rows for x in r], dtype=torch.int32))
+    C, _, st = gpu_colors(g2, 2, gcb.MAXMIN, mode=gcb.MODE_COUNT)
+    assert (C == ref).all() and st.mode_used == gcb.MODE_COUNT
+    C, _, st = gpu_colors(g2, 2, gcb.LUBY_MIS)
+    assert (C == O.color_luby(g, 2)).all() and st.mode_used == gcb.MODE_COUNT
 
 
 def test_schedule_invariance_and_device_output():
