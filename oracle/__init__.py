@@ -17,6 +17,10 @@ Parity status per function:
                       property per frontier, properness)
   color_hash_is       pinned (golden at T = 0/1/4, K_n closed form, row-order
                       invariance, properness, progress bound R <= 2n+2)
+  ldf (all of the above but Hash IS, reading R21)
+                      pinned (literal Alg.5 with (degree, weight) tuple keys,
+                      LDF greedy = JP closed form, longest-path DP, star and
+                      regular-graph closed forms, certificates with mutations)
   paper-value parity  unpinned: the paper prints no colour count or worked
                       example for any variant (Fig.1b/3 unreadable).
 """
@@ -58,21 +62,21 @@ def lib():
         L.orc_hash_key.argtypes, L.orc_hash_key.restype = [u64, i32], u32
         L.orc_priority.argtypes, L.orc_priority.restype = [u64, i32, u32], u32
         L.orc_priorities.argtypes, L.orc_priorities.restype = [u64, i32, i64, P], None
-        L.orc_color_maxmin.argtypes = [i64, P, P, u64, i32, P, P, i64, i64]
+        L.orc_color_maxmin.argtypes = [i64, P, P, u64, i32, P, P, i64, i64, i32]
         L.orc_color_maxmin.restype = i64
-        L.orc_color_luby.argtypes, L.orc_color_luby.restype = [i64, P, P, u64, P, P], i64
-        L.orc_color_is_alg2.argtypes, L.orc_color_is_alg2.restype = [i64, P, P, u64, P, P], i64
-        L.orc_color_jp_alg4.argtypes, L.orc_color_jp_alg4.restype = [i64, P, P, u64, P, P], i64
+        L.orc_color_luby.argtypes, L.orc_color_luby.restype = [i64, P, P, u64, P, P, i32], i64
+        L.orc_color_is_alg2.argtypes, L.orc_color_is_alg2.restype = [i64, P, P, u64, P, P, i32], i64
+        L.orc_color_jp_alg4.argtypes, L.orc_color_jp_alg4.restype = [i64, P, P, u64, P, P, i32], i64
         L.orc_color_hash_is.argtypes = [i64, P, P, u64, i32, P, P]
         L.orc_color_hash_is.restype = i64
         L.orc_color_greedy.argtypes, L.orc_color_greedy.restype = [i64, P, P, P, P], i64
-        L.orc_color_greedy_by_priority.argtypes = [i64, P, P, u64, P]
+        L.orc_color_greedy_by_priority.argtypes = [i64, P, P, u64, P, i32]
         L.orc_color_greedy_by_priority.restype = i64
         L.orc_check_proper.argtypes, L.orc_check_proper.restype = [i64, P, P, P], i64
         L.orc_count_colors.argtypes, L.orc_count_colors.restype = [i64, P], i64
         L.orc_compact_colors.argtypes, L.orc_compact_colors.restype = [i64, P], i64
-        L.orc_cert_maxmin.argtypes, L.orc_cert_maxmin.restype = [i64, P, P, u64, i32, P], i64
-        L.orc_cert_mex.argtypes, L.orc_cert_mex.restype = [i64, P, P, u64, P], i64
+        L.orc_cert_maxmin.argtypes, L.orc_cert_maxmin.restype = [i64, P, P, u64, i32, P, i32], i64
+        L.orc_cert_mex.argtypes, L.orc_cert_mex.restype = [i64, P, P, u64, P, i32], i64
         L.orc_num_threads.argtypes, L.orc_num_threads.restype = [], i32
         L.orc_set_threads.argtypes, L.orc_set_threads.restype = [i32], None
         _lib = L
@@ -127,14 +131,16 @@ class OracleError(RuntimeError):
 
 
 def color_maxmin(g, seed: int, H: int = 1, max_rounds: int = 1 << 40,
-                 with_stats: bool = False):
+                 with_stats: bool = False, ldf: bool = False):
     """Max-min (H=1) / multi-hash (H>1) IS colouring, Alg.1 + Alg.5 with snapshot
-    semantics. Returns uint32 raw colours (and (rounds, N_k list) if with_stats)."""
+    semantics. Returns uint32 raw colours (and (rounds, N_k list) if with_stats).
+    ldf: priorities (degree, weight), largest degree first (R21)."""
     n, ro, ci = _csr(g)
     C = np.empty(max(n, 1), dtype=np.uint32)
     cap = 1 << 16
     nk = np.zeros(cap, dtype=np.int64)
-    r = lib().orc_color_maxmin(n, _pp(ro), _p(ci), seed, H, _pp(C), _pp(nk), cap, max_rounds)
+    r = lib().orc_color_maxmin(n, _pp(ro), _p(ci), seed, H, _pp(C), _pp(nk), cap, max_rounds,
+                               int(ldf))
     if r < 0:
         raise OracleError(f"orc_color_maxmin failed: {r}")
     C = C[:n]
@@ -143,12 +149,12 @@ def color_maxmin(g, seed: int, H: int = 1, max_rounds: int = 1 << 40,
     return C
 
 
-def color_luby(g, seed: int, with_stats: bool = False):
+def color_luby(g, seed: int, with_stats: bool = False, ldf: bool = False):
     """Luby MIS colouring, Alg.2 outer + Alg.3 inner loop, fixed weights."""
     n, ro, ci = _csr(g)
     C = np.empty(max(n, 1), dtype=np.uint32)
     inner = np.zeros(1, dtype=np.int64)
-    r = lib().orc_color_luby(n, _pp(ro), _p(ci), seed, _pp(C), _pp(inner))
+    r = lib().orc_color_luby(n, _pp(ro), _p(ci), seed, _pp(C), _pp(inner), int(ldf))
     if r < 0:
         raise OracleError(f"orc_color_luby failed: {r}")
     if with_stats:
@@ -156,24 +162,24 @@ def color_luby(g, seed: int, with_stats: bool = False):
     return C[:n]
 
 
-def _alg2(fn, g, seed, with_stats):
+def _alg2(fn, g, seed, with_stats, ldf=False):
     n, ro, ci = _csr(g)
     C = np.empty(max(n, 1), dtype=np.uint32)
     rounds = np.zeros(1, dtype=np.int64)
-    r = fn(n, _pp(ro), _p(ci), seed, _pp(C), _pp(rounds))
+    r = fn(n, _pp(ro), _p(ci), seed, _pp(C), _pp(rounds), int(ldf))
     if r < 0:
         raise OracleError(f"{fn.__name__} failed: {r}")
     return (C[:n], int(rounds[0])) if with_stats else C[:n]
 
 
-def color_is_alg2(g, seed: int, with_stats: bool = False):
+def color_is_alg2(g, seed: int, with_stats: bool = False, ldf: bool = False):
     """Max-only IS colouring, Alg.2 as written (colour = iteration)."""
-    return _alg2(lib().orc_color_is_alg2, g, seed, with_stats)
+    return _alg2(lib().orc_color_is_alg2, g, seed, with_stats, ldf)
 
 
-def color_jp_alg4(g, seed: int, with_stats: bool = False):
+def color_jp_alg4(g, seed: int, with_stats: bool = False, ldf: bool = False):
     """GraphBLAS Jones-Plassmann, Alg.2 with Alg.4's frontier colour."""
-    return _alg2(lib().orc_color_jp_alg4, g, seed, with_stats)
+    return _alg2(lib().orc_color_jp_alg4, g, seed, with_stats, ldf)
 
 
 def color_hash_is(g, seed: int, table: int, with_stats: bool = False):
@@ -198,11 +204,11 @@ def color_greedy(g, order=None):
     return C[:n]
 
 
-def color_greedy_by_priority(g, seed: int):
+def color_greedy_by_priority(g, seed: int, ldf: bool = False):
     """First-fit greedy in descending p_0 order (closed form of Luby, R10)."""
     n, ro, ci = _csr(g)
     C = np.empty(max(n, 1), dtype=np.uint32)
-    r = lib().orc_color_greedy_by_priority(n, _pp(ro), _p(ci), seed, _pp(C))
+    r = lib().orc_color_greedy_by_priority(n, _pp(ro), _p(ci), seed, _pp(C), int(ldf))
     if r < 0:
         raise OracleError(f"orc_color_greedy_by_priority failed: {r}")
     return C[:n]
@@ -225,16 +231,16 @@ def compact_colors(C) -> np.ndarray:
     return C
 
 
-def cert_maxmin(g, seed: int, H: int, C) -> int:
+def cert_maxmin(g, seed: int, H: int, C, ldf: bool = False) -> int:
     n, ro, ci = _csr(g)
     C = np.ascontiguousarray(C, dtype=np.uint32)
-    return int(lib().orc_cert_maxmin(n, _pp(ro), _p(ci), seed, H, _p(C)))
+    return int(lib().orc_cert_maxmin(n, _pp(ro), _p(ci), seed, H, _p(C), int(ldf)))
 
 
-def cert_mex(g, seed: int, C) -> int:
+def cert_mex(g, seed: int, C, ldf: bool = False) -> int:
     n, ro, ci = _csr(g)
     C = np.ascontiguousarray(C, dtype=np.uint32)
-    return int(lib().orc_cert_mex(n, _pp(ro), _p(ci), seed, _p(C)))
+    return int(lib().orc_cert_mex(n, _pp(ro), _p(ci), seed, _p(C), int(ldf)))
 
 
 def num_threads() -> int:

@@ -1724,13 +1724,18 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
     cudaStream_t st = g->stream;
     GC_CUDA_TRY(cudaMemsetAsync(s.cctr, 0, kCCtrWords * sizeof(unsigned long long), st));
     const bool prof = p.prof && p.prof->on;
+    // the counting pass and the persistent kernel are bracketed by events on
+    // every colouring (un-instrumented kernels: gc_stats kernel_ms[1] / [0])
+    EventPair ev01;
     cudaEvent_t e0 = nullptr, e1 = nullptr, e2 = nullptr;
-    if (prof) {
-        GC_CUDA_TRY(cudaEventCreate(&e0));
-        GC_CUDA_TRY(cudaEventCreate(&e1));
-        GC_CUDA_TRY(cudaEventCreate(&e2));
-        GC_CUDA_TRY(cudaEventRecord(e0, st));
-    }
+    GC_CUDA_TRY(cudaEventCreate(&ev01.e0));
+    GC_CUDA_TRY(cudaEventCreate(&ev01.e1));
+    e0 = ev01.e0;
+    e1 = ev01.e1;
+    EventPair ev2;
+    GC_CUDA_TRY(cudaEventCreate(&ev2.e0));
+    e2 = ev2.e0;
+    GC_CUDA_TRY(cudaEventRecord(e0, st));
     const uint32_t key = p.keys.k[0];
     unsigned long long *nhubs = s.cctr + cHubs;
     {
@@ -1755,7 +1760,7 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
         }
         GC_CUDA_TRY(cudaGetLastError());
     }
-    if (prof) GC_CUDA_TRY(cudaEventRecord(e1, st));
+    GC_CUDA_TRY(cudaEventRecord(e1, st));
     CArgs a;
     a.ro = g->ro;
     a.ci = g->ci;
@@ -1806,7 +1811,7 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
     else rc = prof ? launch<true, false, false>(g, a, &blocks) : launch<false, false, false>(g, a, &blocks);
     if (rc) return rc;
     r->launches += 3;  // k_count, k_count_hub, persistent kernel
-    if (prof) GC_CUDA_TRY(cudaEventRecord(e2, st));
+    GC_CUDA_TRY(cudaEventRecord(e2, st));
     unsigned long long h[kCCtrWords];
     GC_CUDA_TRY(cudaMemcpyAsync(h, s.cctr, sizeof(h), cudaMemcpyDeviceToHost, st));
     GC_CUDA_TRY(cudaStreamSynchronize(st));
@@ -1831,20 +1836,20 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
     }
     r->rounds = (int64_t)h[cRounds];
     r->inner = r->rounds;
-    if (prof) {
+    if (p.prof) {
+        // class 0: the persistent kernel; 1: counting kernels (both timed on
+        // every colouring); PROF only: 2 its init phase (round 0), 3 its
+        // rounds (globaltimer, block 0), algorithmic bytes
         float ms_all = 0.f, ms_cnt = 0.f;
         cudaEventElapsedTime(&ms_all, e0, e2);
         cudaEventElapsedTime(&ms_cnt, e0, e1);
-        cudaEventDestroy(e0);
-        cudaEventDestroy(e1);
-        cudaEventDestroy(e2);
-        // class 0: the persistent kernel; 1: counting kernels; 2: its init
-        // phase (round 0); 3: its rounds (globaltimer, block 0)
         p.prof->ms[0] += ms_all - ms_cnt;
         p.prof->launches[0] += 1;
         p.prof->launch_us.push_back(1e3f * (ms_all - ms_cnt));
         p.prof->ms[1] += ms_cnt;
         p.prof->launches[1] += 2;
+    }
+    if (prof) {
         p.prof->ms[2] += (double)h[cPhaseNs] / 1e6;
         p.prof->ms[3] += (double)h[cPhaseNs + 1] / 1e6;
         // algorithmic bytes.  Counting: 8 B offsets + 8 B

@@ -517,6 +517,28 @@ def test_cfg5_style_partitioned_rmat_s25():
     assert O.cert_maxmin(gh, 1, 1, C) == 0
 
 
+@pytest.mark.parametrize("scale", [16, 20])
+def test_rgg_workloads_all_variants(scale):
+    """the random geometric graphs of the paper's scaling study
+    (rgg_n_2_<scale>, Table I, Fig.3) -- every variant
+    element by element against the oracle (rounds too, where defined), in the
+    launch configuration AUTO picks."""
+    g = G.rgg(scale, seed=1, device="cuda").to("cpu")
+    cases = [("maxmin", 1), ("multihash", 4), ("luby", 1), ("is_alg2", 1), ("jp_alg4", 1),
+             ("hash_is8", 1)]
+    for vname, H in cases:
+        C, k, st = gpu_colors(g, 1, variant_of(vname, H), frontier_cap=4096)
+        ref = oracle_colors(g, 1, vname, H)
+        assert (C == ref).all(), vname
+        assert k == O.count_colors(ref), vname
+        if vname in ("maxmin", "multihash"):
+            _, R, nk = O.color_maxmin(g, 1, H, with_stats=True)
+            assert st.rounds == R and st.frontier_sizes == nk
+        if vname in ("is_alg2", "jp_alg4"):
+            _, R = (O.color_is_alg2 if vname == "is_alg2" else O.color_jp_alg4)(g, 1, with_stats=True)
+            assert st.rounds == R
+
+
 def test_cfg5_rmat_s27_one_gpu_and_partitions():
     """cfg5 at its stated size: R-MAT s27 ef16 (1.3e8 vertices, nnz > 2^31).
     One B200 colours it through gc_create_csr / AUTO (the bench launch

@@ -45,14 +45,21 @@ def fmix32_inverse(h: int) -> int:
     return h
 
 
-def alg5_literal(n, adj, seed, H, rng):
+def ldf_key(adj, seed):
+    """R21 restated with Python tuples: priority of v under hash j is
+    (deg(v), p_j(v)), compared lexicographically (largest degree first)."""
+    return lambda j, v: (len(adj[v]), O.priority(seed, j, v))
+
+
+def alg5_literal(n, adj, seed, H, rng, key=None):
     """PAPER.md Algorithm 5 transcribed line by line, 1-based colours, IN PLACE,
     threads in a random order each iteration (the GPU's nondeterministic
     schedule).  Generalised to H hashes by letting hash j of an iteration use
     colour = 2*(iteration*H + j); the L26 test skips u iff C[u] is valid and not
     one of this iteration's colours.  Returns 0-based colours (paper - 1)."""
     INVALID = 0
-    R = [[O.priority(seed, j, v) for v in range(n)] for j in range(H)]  # L7
+    key = key or (lambda j, v: O.priority(seed, j, v))
+    R = [[key(j, v) for v in range(n)] for j in range(H)]                 # L7
     C = [INVALID] * n                                                      # L5
     iteration = 0                                                          # L3
     while any(c == INVALID for c in C):                                    # L9
@@ -85,11 +92,12 @@ def alg5_literal(n, adj, seed, H, rng):
     return [c - 1 for c in C], iteration
 
 
-def jones_plassmann(n, adj, seed):
+def jones_plassmann(n, adj, seed, key=None):
     """Jones-Plassmann: a vertex colours itself with the smallest
     colour unused by its neighbours once every higher-weight neighbour is
     coloured.  Synchronous rounds."""
-    p = [O.priority(seed, 0, v) for v in range(n)]
+    key = key or (lambda j, v: O.priority(seed, j, v))
+    p = [key(0, v) for v in range(n)]
     C = [None] * n
     while any(c is None for c in C):
         ready = [v for v in range(n) if C[v] is None and
@@ -281,13 +289,14 @@ def test_hash_is_large_table_reuses_colours():
 
 
 # ------------------------------------------------ Alg.2 / Alg.4
-def _longest_decreasing_path(g, seed):
+def _longest_decreasing_path(g, seed, key=None):
     # length (in vertices) of the longest strictly-decreasing-weight path
     # ending at each vertex: DP over vertices in decreasing weight order
-    p = [O.priority(seed, 0, v) for v in range(g.n)]
     adj = adjacency(g)
+    key = key or (lambda j, v: O.priority(seed, j, v))
+    p = [key(0, v) for v in range(g.n)]
     depth = [0] * g.n
-    for v in sorted(range(g.n), key=lambda x: -p[x]):
+    for v in sorted(range(g.n), key=lambda x: p[x], reverse=True):
         depth[v] = 1 + max((depth[u] for u in adj[v] if p[u] > p[v]), default=0)
     return depth
 
@@ -508,3 +517,79 @@ def test_oracle_rejects_self_loops():
                                                                                   dtype=__import__("torch").int32))
     with pytest.raises(O.OracleError):
         O.color_maxmin(g, 1)
+
+
+# ------------------------------------------ N4: largest-degree-first (R21)
+@pytest.mark.parametrize("H", [1, 2])
+def test_ldf_maxmin_equals_literal_alg5_with_degree_keys(H):
+    """LDF max-min = Alg.5 transcribed literally (in place, random thread
+    order) with the priority replaced by the (degree, weight) tuple."""
+    rng = random.Random(40 + H)
+    for g in random_graphs(50, 30, seed0=60 + H):
+        adj = adjacency(g)
+        for seed in (2, 9):
+            lit, iters = alg5_literal(g.n, adj, seed, H, rng, key=ldf_key(adj, seed))
+            C, R, _ = O.color_maxmin(g, seed, H, with_stats=True, ldf=True)
+            assert C.tolist() == lit and R == iters
+            assert O.cert_maxmin(g, seed, H, C, ldf=True) == 0
+            assert O.check_proper(g, C) == 0
+
+
+def test_ldf_luby_alg2_alg4_closed_forms():
+    """LDF Luby = first-fit greedy in decreasing (degree, weight) order (the
+    classic largest-degree-first greedy) = Jones-Plassmann with those keys;
+    LDF Alg.2 colour = longest decreasing-(degree, weight) path - 1; the mex
+    certificate with LDF keys accepts them."""
+    for g in random_graphs(60, 35, seed0=71):
+        adj = adjacency(g)
+        key = ldf_key(adj, 3)
+        order = sorted(range(g.n), key=lambda v: key(0, v), reverse=True)
+        C = O.color_luby(g, 3, ldf=True)
+        assert C.tolist() == first_fit(g.n, adj, order) == jones_plassmann(g.n, adj, 3, key=key)
+        assert (O.color_greedy_by_priority(g, 3, ldf=True) == C).all()
+        assert O.cert_mex(g, 3, C, ldf=True) == 0
+        C2, R2 = O.color_is_alg2(g, 3, with_stats=True, ldf=True)
+        d = _longest_decreasing_path(g, 3, key=key)
+        assert C2.tolist() == [x - 1 for x in d] and R2 == (max(d) if g.n else 0)
+        C4 = O.color_jp_alg4(g, 3, ldf=True)
+        assert O.check_proper(g, C4) == 0
+
+
+def test_ldf_closed_forms_star_and_regular_graphs():
+    """Star K_{1,s}: the centre has the largest degree, so under LDF it is the
+    round-0 local max (colour 0) and every leaf a local min (colour 1), for
+    every seed; Luby LDF colours the centre 0 and the leaves 1.  On regular
+    graphs (cycle, K_n, hypercube) every degree ties, so LDF equals the plain
+    random-priority colouring."""
+    s = 40
+    star = G.csr_from_lists(s + 1, [(0, i) for i in range(1, s + 1)])
+    for seed in range(1, 8):
+        assert O.color_maxmin(star, seed, ldf=True).tolist() == [0] + [1] * s
+        assert O.color_luby(star, seed, ldf=True).tolist() == [0] + [1] * s
+    d = 5
+    cube = G.csr_from_lists(1 << d, [(v, v ^ (1 << b)) for v in range(1 << d) for b in range(d)
+                                     if v < v ^ (1 << b)])
+    for g in (G.csr_from_lists(9, [(i, (i + 1) % 9) for i in range(9)]),
+              G.csr_from_lists(8, [(a, b) for a in range(8) for b in range(a + 1, 8)]), cube):
+        for seed in (1, 4):
+            assert (O.color_maxmin(g, seed, ldf=True) == O.color_maxmin(g, seed)).all()
+            assert (O.color_luby(g, seed, ldf=True) == O.color_luby(g, seed)).all()
+            assert (O.color_jp_alg4(g, seed, ldf=True) == O.color_jp_alg4(g, seed)).all()
+
+
+def test_ldf_certificates_reject_mutations():
+    rng = random.Random(77)
+    for g in random_graphs(25, 40, seed0=81):
+        C = O.color_maxmin(g, 6, ldf=True)
+        L = O.color_luby(g, 6, ldf=True)
+        assert O.cert_maxmin(g, 6, 1, C, ldf=True) == 0 and O.cert_mex(g, 6, L, ldf=True) == 0
+        for _ in range(10):
+            v = rng.randrange(g.n)
+            D = C.copy()
+            D[v] = (int(D[v]) + rng.randrange(1, 4)) % (int(C.max()) + 3)
+            if D[v] != C[v]:
+                assert O.cert_maxmin(g, 6, 1, D, ldf=True) != 0
+            E = L.copy()
+            E[v] = (int(E[v]) + rng.randrange(1, 4)) % (int(L.max()) + 3)
+            if E[v] != L[v]:
+                assert O.cert_mex(g, 6, E, ldf=True) != 0
