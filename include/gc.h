@@ -94,6 +94,14 @@ typedef enum gc_status {
 #define GC_HASH_TABLE_MAX 64
 #define GC_VARIANT_KIND(v) ((v) & 0xFF)
 #define GC_VARIANT_HASHES(v) (((v) >> 8) & 0xFF)
+/* GC_LDF(v): largest-degree-first priorities (PAPER.md:1090-1098,
+ *   reading R21): the weight of v becomes the pair (deg(v), p(v)), compared
+ *   lexicographically (the larger degree wins, the seeded weight breaks
+ *   ties; deg = number of distinct neighbours).  Applies to GC_MAXMIN,
+ *   GC_LUBY_MIS, GC_IS_ALG2 and GC_JP_ALG4; COUNT mode, single GPU.  An
+ *   asymmetric adjacency returns GC_ERR_NOT_SYMMETRIC (no fallback). */
+#define GC_LDF(v) ((v) | (1 << 16))
+#define GC_VARIANT_LDF(v) (((v) >> 16) & 1)
 
 /* ---------------------------------------------------------------- flags */
 #define GC_BORROW_DEVICE (1u << 0) /* create: adopt device CSR pointers without

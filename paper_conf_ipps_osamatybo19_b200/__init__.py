@@ -36,6 +36,12 @@ def MULTIHASH(h: int) -> int:
 HASH_TABLE_MAX = 64
 
 
+def LDF(variant: int) -> int:
+    """Largest-degree-first priorities (reading R21) for GC_MAXMIN,
+    GC_LUBY_MIS, GC_IS_ALG2 and GC_JP_ALG4."""
+    return variant | (1 << 16)
+
+
 def HASH_IS(t: int) -> int:
     """The paper's Hash IS (Alg.6, deterministic readings R16-R20), table of t colours."""
     return 5 | (t << 8)

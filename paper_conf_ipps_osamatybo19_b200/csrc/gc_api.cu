@@ -352,6 +352,7 @@ static void free_scratch(Scratch &s) {
     dfree(s.hubs);
     dfree(s.cctr);
     dfree(s.jslot);
+    dfree(s.deg);
     dfree(s.jcr);
     dfree(s.cM);
     dfree(s.crow);
@@ -536,8 +537,21 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
         set_error("gc_color_ex: unknown mode");
         return GC_ERR_INVALID_ARG;
     }
+    const int ldf = GC_VARIANT_LDF(o->variant) ? 1 : 0;
+    if ((o->variant & ~(0xFFFF | GC_LDF(0))) != 0 ||
+        (ldf && (kind == GC_MULTIHASH(0) || kind == GC_HASH_IS(0)))) {
+        set_error("gc_color_ex: bad variant flags (GC_LDF applies to GC_MAXMIN, GC_LUBY_MIS, GC_IS_ALG2, "
+                  "GC_JP_ALG4)");
+        return GC_ERR_INVALID_ARG;
+    }
     GC_CUDA_TRY(cudaSetDevice(g->device));
-    if (g->dist) return gc_color_dist(g, o, colors_out, stats);
+    if (g->dist) {
+        if (ldf) {
+            set_error("gc_color_ex: GC_LDF is single-GPU only");
+            return GC_ERR_INVALID_ARG;
+        }
+        return gc_color_dist(g, o, colors_out, stats);
+    }
 
     const bool luby = kind == GC_LUBY_MIS;
     // Alg.2 as written / Alg.2 + Alg.4: COUNT mode only
@@ -557,6 +571,7 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     // 0.58; 117^3: 0.43 vs 0.47), whose few uniform rounds stream the CSR.
     if (mode == GC_MODE_AUTO)
         mode = (luby || g->max_deg > 8 || g->n < (1 << 20)) ? GC_MODE_COUNT : GC_MODE_SWEEP;
+    if (ldf) mode = GC_MODE_COUNT;  // (degree, weight) keys: COUNT kernels only
     if (luby && mode != GC_MODE_COUNT) mode = GC_MODE_SWEEP;
     if (H != 1 && mode != GC_MODE_COUNT) mode = GC_MODE_SWEEP;  // multi-hash: SWEEP or COUNT
 
@@ -570,9 +585,14 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     p.eval_big_min = o->hub_deg_min > 0 ? o->hub_deg_min : 256;
     p.batch_rounds = o->batch_rounds;
     p.max_rounds = (int64_t)(0x7FFFFFFFll / (2 * H)) + 1;
+    p.ldf = ldf;
     Profile prof;
     prof.on = (o->flags & GC_PROFILE) != 0;
     p.prof = &prof;
+    if (ldf) {  // the degree of R21 is the number of distinct neighbours
+        rc = ensure_strict_rows(g);
+        if (rc) return rc;
+    }
 
     EventPair ev;  // destroyed on every exit path
     GC_CUDA_TRY(cudaEventCreate(&ev.e0));
@@ -610,13 +630,13 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
         if (!rc) rc = run_count_variant();
         else if (rc == GC_ERR_OOM || rc == GC_ERR_TOO_LARGE) rc = GC_ERR_NOT_SYMMETRIC;  // no copy: fall back
     }
-    if (rc == GC_ERR_TOO_LARGE && mode == GC_MODE_COUNT && jpv < 2) {
+    if (rc == GC_ERR_TOO_LARGE && mode == GC_MODE_COUNT && jpv < 2 && !ldf) {
         // a round's item count overflowed the persistent kernel's round word
         // (gc_count.cu, trap 9): the EVENT / SWEEP kernels have no such field
         g->count_unsafe = true;
         rc = GC_ERR_NOT_SYMMETRIC;
     }
-    if (rc == GC_ERR_NOT_SYMMETRIC && mode == GC_MODE_COUNT && jpv < 2) {
+    if (rc == GC_ERR_NOT_SYMMETRIC && mode == GC_MODE_COUNT && jpv < 2 && !ldf) {
         // Still asymmetric after deduplication: the adjacency SETS are not
         // symmetric (a count underflow or a stall -- never a silently wrong
         // colour).  The witness / sweep kernels test the set

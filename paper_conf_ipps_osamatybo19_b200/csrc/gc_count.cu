@@ -162,7 +162,16 @@ struct CArgs {
     uint32_t bwords;
     int H;                         // MH: weight functions (count words v * H + j)
     uint32_t mkeys[GC_MAX_HASHES]; // MH: their keys K_j
+    const uint32_t *dg;            // LDF: vertex degrees; nullptr = weights only
 };
+
+// Priority key of v (R1; with LDF the (degree, weight) pair of R21 as one
+// 64-bit integer, degree in the high half): comparisons of keys are the
+// comparisons of Alg.5 L29-34 / Alg.2 L9.
+__device__ __forceinline__ uint64_t prio_key(const CArgs &a, uint32_t v) {
+    const uint64_t w = weight_mix(v ^ a.key);
+    return a.dg ? w | ((uint64_t)__ldg(a.dg + v) << 32) : w;
+}
 // JP mex slot of a long row: a 1024-bit presence set of its predecessors'
 // colours + the number of its entries not yet walked (the segment that takes
 // it to zero computes the mex and writes the colour).
@@ -494,7 +503,7 @@ __device__ __forceinline__ void clear_status(const CArgs &a, uint32_t v) {
 // set: bits < 64 of `mask` (short rows), or bits < 1024 of the warp's shared
 // bitmap `sbits` (WIDE: long-row segments).  mex = `want_mex` lanes only.
 template <int Q, bool JP = false, bool WIDE = false>
-__device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, int64_t e,
+__device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint64_t pv, int64_t e,
                                      int64_t end, int stride, uint32_t k, uint32_t &nvis,
                                      unsigned long long *mask = nullptr, uint32_t *sbits = nullptr,
                                      bool want_mex = false, bool want_set = false,
@@ -532,7 +541,8 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint32_t pv, in
     for (int q = 0; q < Q; ++q) {
         const bool live = w[q] != kNone;
         const uint32_t wq = live ? w[q] : 0u;
-        hi[q] = live && pv > weight_mix(wq ^ a.key);  // v is a larger neighbour of w
+        // v is a larger neighbour of w (LDF: the degree decides first, R21)
+        hi[q] = live && pv > ((uint64_t)weight_mix(wq ^ a.key) | (a.dg ? (uint64_t)__ldg(a.dg + wq) << 32 : 0ull));
         cv[q] = kNone;
 #if GC_PACKED
         slot[q] = (live && a.nbig > 0) ? big_slot(wq) : -1;
@@ -880,9 +890,9 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
 // predecessors' colours into the warp's window `sb`; merge it into v's slot
 // and retire its entries; the segment that retires the last entry computes
 // the mex and colours v (first-fit, R10).
-__device__ __noinline__ uint32_t jp_mex_rescan(const CArgs &a, uint32_t v, uint32_t pv, uint32_t *sb);
+__device__ __noinline__ uint32_t jp_mex_rescan(const CArgs &a, uint32_t v, uint64_t pv, uint32_t *sb);
 
-__device__ __forceinline__ void jp_segment_done(const CArgs &a, uint32_t v, uint32_t len, uint32_t pv,
+__device__ __forceinline__ void jp_segment_done(const CArgs &a, uint32_t v, uint32_t len, uint64_t pv,
                                                 uint32_t *sb, uint32_t k) {
     const unsigned lane = lane_id();
     __syncwarp();
@@ -920,7 +930,7 @@ __device__ __forceinline__ void jp_segment_done(const CArgs &a, uint32_t v, uint
 
 // mex >= kMexWin (a vertex with >= 1024 predecessors of distinct colours):
 // the warp rescans the row for successive 1024-colour windows (rare).
-__device__ __noinline__ uint32_t jp_mex_rescan(const CArgs &a, uint32_t v, uint32_t pv, uint32_t *sb) {
+__device__ __noinline__ uint32_t jp_mex_rescan(const CArgs &a, uint32_t v, uint64_t pv, uint32_t *sb) {
     const unsigned lane = lane_id();
     const int64_t rs = a.ro[v], re = a.ro[v + 1];
     for (uint32_t b = kMexWin;; b += kMexWin) {
@@ -929,7 +939,7 @@ __device__ __noinline__ uint32_t jp_mex_rescan(const CArgs &a, uint32_t v, uint3
         __syncwarp();
         for (int64_t e = rs + lane; e < re; e += 32) {
             const uint32_t u = a.ci[e];
-            if (weight_mix(u ^ a.key) > pv) {
+            if (prio_key(a, u) > pv) {
                 const uint32_t c = __ldcg(a.C + u) - b;
                 if (c < kMexWin) atomicOr(sb + (c >> 5), 1u << (c & 31u));
             }
@@ -1139,7 +1149,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                 // longer rows: one <= kSeg-entry item per warp
                 Item it = a.WL[wl0 + u];
                 if (it.v == kNone) it.lf = 0;  // hole left by schedule_fresh
-                const uint32_t pv = weight_mix(it.v ^ a.key);
+                const uint64_t pv = prio_key(a, it.v);
                 if (JP && a.jpv != 1) {  // Alg.2 / Alg.4: the colour is the round (remapped for Alg.4)
                     if ((it.lf & kFirst) && lane == 0) {
                         a.C[it.v] = k;
@@ -1159,7 +1169,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                     const uint32_t z = cl ? __ldcg(a.Zlo + it.v) : 0u;
                     long long tp[3] = {0, 0, 0};
                     if (GC_PROF_UNIT && prs) {
-                        asm volatile("" ::"r"(pv));
+                        asm volatile("" ::"l"(pv));
                         tp[2] = clock64();
                     }
                     if (MH)
@@ -1185,7 +1195,8 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
             } else if (lane_rows) {
                 // short rows: one per lane, 4 entries per step
                 const unsigned long long idx = sl0 + 32 * (u - nw) + lane;
-                uint32_t v = kNone, len = 0, pv = 0;
+                uint32_t v = kNone, len = 0;
+                uint64_t pv = 0;
                 int64_t e0 = 0;
                 bool want = false, cl = false;
                 uint32_t lf = 0, z = 0;
@@ -1195,7 +1206,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                     lf = it.lf;
                     len = it.lf & kLenMask;
                     e0 = it.e0;
-                    pv = weight_mix(v ^ a.key);
+                    pv = prio_key(a, v);
                     want = JP && a.jpv == 1 && (it.lf & kFirst);
                     if (JP && a.jpv != 1 && (it.lf & kFirst)) {
                         a.C[v] = k;
@@ -1218,7 +1229,8 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
             } else {
                 // short rows: 4 per warp, 8 lanes each, 4 entries per lane
                 const unsigned long long idx = sl0 + 4 * (u - nw) + (lane >> 3);
-                uint32_t v = kNone, len = 0, pv = 0;
+                uint32_t v = kNone, len = 0;
+                uint64_t pv = 0;
                 int64_t e0 = 0;
                 bool want = false, cl = false;
                 uint32_t lf = 0, z = 0;
@@ -1228,7 +1240,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                     lf = it.lf;
                     len = it.lf & kLenMask;
                     e0 = it.e0;
-                    pv = weight_mix(v ^ a.key);
+                    pv = prio_key(a, v);
                     want = JP && a.jpv == 1 && (it.lf & kFirst);
                     if (JP && a.jpv != 1 && (it.lf & kFirst) && (lane & 7u) == 0u) {
                         a.C[v] = k;
@@ -1326,11 +1338,18 @@ struct CountKeys {
     int H;
 };
 
+// LDF (dg != nullptr, H = 1): the key of R21, (degree, weight), decides
+__device__ __forceinline__ uint64_t ckey(const uint32_t *dg, uint32_t v, uint32_t key) {
+    const uint64_t w = weight_mix(v ^ key);
+    return dg ? w | ((uint64_t)__ldg(dg + v) << 32) : w;
+}
+
 template <bool MH>
 __global__ void __launch_bounds__(256) k_count(const int64_t *__restrict__ ro,
                                                const uint32_t *__restrict__ ci, int64_t n,
                                                CountKeys keys, unsigned long long *cnt,
-                                               uint2 *hubs, unsigned long long *nhubs, int jp) {
+                                               uint2 *hubs, unsigned long long *nhubs, int jp,
+                                               const uint32_t *__restrict__ dg) {
     const unsigned lane = lane_id();
     const unsigned long long gw = ((unsigned long long)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const unsigned long long nw = ((unsigned long long)gridDim.x * blockDim.x) >> 5;
@@ -1350,10 +1369,10 @@ __global__ void __launch_bounds__(256) k_count(const int64_t *__restrict__ ro,
             for (int q = 0; q < 16; ++q) u[q] = q < deg ? __ldcs(ci + rs + q) : 0u;
             for (int j = 0; j < H; ++j) {
                 const uint32_t key = keys.k[j];
-                const uint32_t pv = weight_mix((uint32_t)v ^ key);
+                const uint64_t pv = ckey(MH ? nullptr : dg, (uint32_t)v, key);
                 uint32_t h = 0;
 #pragma unroll
-                for (int q = 0; q < 16; ++q) h += (q < deg && weight_mix(u[q] ^ key) > pv) ? 1u : 0u;
+                for (int q = 0; q < 16; ++q) h += (q < deg && ckey(MH ? nullptr : dg, u[q], key) > pv) ? 1u : 0u;
                 cnt[(size_t)v * H + j] = ((unsigned long long)h << 32) | (unsigned long long)(jp ? 1 : deg - h);
             }
         }
@@ -1373,7 +1392,7 @@ __global__ void __launch_bounds__(256) k_count(const int64_t *__restrict__ ro,
             const uint32_t vs = (uint32_t)(base + src);
             for (int j = 0; j < H; ++j) {
                 const uint32_t key = keys.k[j];
-                const uint32_t p = weight_mix(vs ^ key);
+                const uint64_t p = ckey(MH ? nullptr : dg, vs, key);
                 uint32_t h = 0;
                 for (int64_t e = r0 + lane; e < r1; e += 128) {
                     uint32_t u[4];
@@ -1381,7 +1400,7 @@ __global__ void __launch_bounds__(256) k_count(const int64_t *__restrict__ ro,
                     for (int q = 0; q < 4; ++q) u[q] = e + 32 * q < r1 ? __ldcs(ci + e + 32 * q) : 0u;
 #pragma unroll
                     for (int q = 0; q < 4; ++q)
-                        h += (e + 32 * q < r1 && weight_mix(u[q] ^ key) > p) ? 1u : 0u;
+                        h += (e + 32 * q < r1 && ckey(MH ? nullptr : dg, u[q], key) > p) ? 1u : 0u;
                 }
                 h = __reduce_add_sync(kFull, h);
                 if (lane == (unsigned)src)
@@ -1398,7 +1417,8 @@ template <bool MH>
 __global__ void __launch_bounds__(256) k_count_hub(const int64_t *__restrict__ ro,
                                                    const uint32_t *__restrict__ ci, CountKeys keys,
                                                    unsigned long long *cnt, const uint2 *hubs,
-                                                   const unsigned long long *nhubs, int jp) {
+                                                   const unsigned long long *nhubs, int jp,
+                                                   const uint32_t *__restrict__ dg) {
     __shared__ uint32_t red[8];
     const unsigned long long nh = *nhubs;
     const int H = MH ? keys.H : 1;
@@ -1409,11 +1429,11 @@ __global__ void __launch_bounds__(256) k_count_hub(const int64_t *__restrict__ r
         const int64_t c0 = rs + (int64_t)hc.y * kHubChunk, c1 = min(re, c0 + (int64_t)kHubChunk);
         for (int j = 0; j < H; ++j) {
             const uint32_t key = keys.k[j];
-            const uint32_t pv = weight_mix(v ^ key);
+            const uint64_t pv = ckey(MH ? nullptr : dg, v, key);
             uint32_t hcount = 0;
 #pragma unroll 4
             for (int64_t e = c0 + threadIdx.x; e < c1; e += blockDim.x)
-                hcount += weight_mix(__ldcs(ci + e) ^ key) > pv ? 1u : 0u;
+                hcount += ckey(MH ? nullptr : dg, __ldcs(ci + e), key) > pv ? 1u : 0u;
             hcount = __reduce_add_sync(kFull, hcount);
             if (lane_id() == 0) red[threadIdx.x >> 5] = hcount;
             __syncthreads();
@@ -1676,6 +1696,22 @@ int ensure_count_scratch(gc_graph *g) {
     return GC_OK;
 }
 
+__global__ void k_degrees(const int64_t *__restrict__ ro, int64_t n, uint32_t *deg) {
+    for (int64_t v = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; v < n; v += (int64_t)gridDim.x * blockDim.x)
+        deg[v] = (uint32_t)min(ro[v + 1] - ro[v], (int64_t)0xFFFFFFFF);
+}
+
+// LDF: deg[v] = row length (rows are strictly increasing here: gc_api runs
+// ensure_strict_rows first, so it is the number of distinct neighbours)
+static int ensure_degrees(gc_graph *g) {
+    Scratch &s = g->s;
+    if (s.deg) return GC_OK;
+    GC_CUDA_TRY(dmalloc(&s.deg, (size_t)std::max<int64_t>(g->n, 1) * 4));
+    if (g->n > 0) k_degrees<<<g->sm_count * 8, 256, 0, g->stream>>>(g->ro, g->n, s.deg);
+    GC_CUDA_TRY(cudaGetLastError());
+    return GC_OK;
+}
+
 // JP mex slots: one per vertex of degree > kShortMax (each is scheduled once)
 static int ensure_jp_scratch(gc_graph *g) {
     Scratch &s = g->s;
@@ -1738,6 +1774,12 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
     GC_CUDA_TRY(cudaEventRecord(e0, st));
     const uint32_t key = p.keys.k[0];
     unsigned long long *nhubs = s.cctr + cHubs;
+    // LDF: the degree array, built once per graph (seed-independent)
+    const uint32_t *dg = nullptr;
+    if (p.ldf) {
+        if ((rc = ensure_degrees(g))) return rc;
+        dg = s.deg;
+    }
     {
         const int64_t warps = (n + 31) / 32;
         const int blocks = (int)std::min<int64_t>((warps + 7) / 8, (int64_t)g->sm_count * 16);
@@ -1746,17 +1788,18 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
         ck.H = p.H;
         for (int j = 0; j < GC_MAX_HASHES; ++j) ck.k[j] = p.keys.k[j];
         if (mh) {
-            k_count<true><<<blocks, 256, 0, st>>>(g->ro, g->ci, n, ck, s.cnt, hubs, nhubs, 0);
-            k_count_hub<true><<<g->sm_count * 8, 256, 0, st>>>(g->ro, g->ci, ck, s.cnt, hubs, nhubs, 0);
-        } else if (kCountStream) {
+            k_count<true><<<blocks, 256, 0, st>>>(g->ro, g->ci, n, ck, s.cnt, hubs, nhubs, 0, nullptr);
+            k_count_hub<true><<<g->sm_count * 8, 256, 0, st>>>(g->ro, g->ci, ck, s.cnt, hubs, nhubs, 0,
+                                                               nullptr);
+        } else if (kCountStream && !dg) {
             const int64_t nch = s.nch;
             k_count_zero<<<g->sm_count, 256, 0, st>>>(g->ro, s.crow, nch, s.cnt, jp ? 1 : 0);
             k_count_stream<<<(int)std::min<int64_t>(nch, (int64_t)g->sm_count * 8), kCT, 0, st>>>(
                 g->ro, g->ci, g->nnz, nch, s.crow, key, s.cnt, jp ? 1 : 0);
         } else {
-            k_count<false><<<blocks, 256, 0, st>>>(g->ro, g->ci, n, ck, s.cnt, hubs, nhubs, jp ? 1 : 0);
+            k_count<false><<<blocks, 256, 0, st>>>(g->ro, g->ci, n, ck, s.cnt, hubs, nhubs, jp ? 1 : 0, dg);
             k_count_hub<false><<<g->sm_count * 8, 256, 0, st>>>(g->ro, g->ci, ck, s.cnt, hubs, nhubs,
-                                                                jp ? 1 : 0);
+                                                                jp ? 1 : 0, dg);
         }
         GC_CUDA_TRY(cudaGetLastError());
     }
@@ -1786,6 +1829,7 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
     a.jslot_cap = (unsigned long long)s.jslot_cap;
     a.H = p.H;
     for (int j = 0; j < GC_MAX_HASHES; ++j) a.mkeys[j] = p.keys.k[j];
+    a.dg = dg;
     a.M = s.cM;
     a.jpv = jpv;
     a.cr = nullptr;

@@ -199,6 +199,8 @@ int dedup_csr(gc_graph *g) {
     g->nnz = base;
     g->owns_csr = true;
     g->deduped = true;
+    dfree(g->s.deg);  // LDF degrees follow the rows
+    g->s.deg = nullptr;
     nro = nullptr;
     nci = nullptr;
 out:

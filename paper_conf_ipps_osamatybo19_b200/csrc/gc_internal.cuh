@@ -77,6 +77,7 @@ struct Scratch {
     uint32_t *cM = nullptr;              // COUNT mode: status bits (1 = uncoloured)
     uint32_t *crow = nullptr;            // COUNT mode: row of each counting chunk's first entry
     int64_t nch = 0;
+    uint32_t *deg = nullptr;             // LDF: row lengths (seed-independent)
     uint32_t *jslot = nullptr;           // JP (Luby-MIS in COUNT mode): mex slots of long rows
     uint32_t *jcr = nullptr;             // Alg.4: round colours + colour sets
     int64_t jcr_words = 0;
@@ -173,6 +174,7 @@ struct RunParams {
     int32_t eval_big_min = 256;  // event mode: remaining scan length sent to a CTA
     int32_t batch_rounds = 0;
     int64_t max_rounds = 0;
+    int ldf = 0;  // (degree, weight) priorities (R21), COUNT kernels only
 };
 
 struct RunResult {

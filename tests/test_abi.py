@@ -107,9 +107,9 @@ def test_argument_errors_need_no_device(libgc):
 
 def test_variant_codes_match_header():
     # the binding's variant codes are the header's macros, evaluated by the C compiler
-    src = ('#include <stdio.h>\n#include "gc.h"\nint main(void){printf("%d %d %d %d %d %d %d\\n",'
+    src = ('#include <stdio.h>\n#include "gc.h"\nint main(void){printf("%d %d %d %d %d %d %d %d\\n",'
            'GC_MAXMIN, GC_LUBY_MIS, GC_MULTIHASH(4), GC_IS_ALG2, GC_JP_ALG4, GC_HASH_IS(8),'
-           'GC_HASH_TABLE_MAX);return 0;}\n')
+           'GC_HASH_TABLE_MAX, GC_LDF(GC_JP_ALG4));return 0;}\n')
     import tempfile
     with tempfile.TemporaryDirectory() as d:
         c, exe = os.path.join(d, "v.c"), os.path.join(d, "v")
@@ -117,7 +117,7 @@ def test_variant_codes_match_header():
         subprocess.check_call(["gcc", "-I" + os.path.join(ROOT, "include"), "-o", exe, c])
         got = [int(x) for x in subprocess.check_output([exe]).split()]
     assert got == [gcb.MAXMIN, gcb.LUBY_MIS, gcb.MULTIHASH(4), gcb.IS_ALG2, gcb.JP_ALG4,
-                   gcb.HASH_IS(8), gcb.HASH_TABLE_MAX]
+                   gcb.HASH_IS(8), gcb.HASH_TABLE_MAX, gcb.LDF(gcb.JP_ALG4)]
 
 
 def test_binding_rejects_short_buffers():

@@ -539,6 +539,74 @@ def test_rgg_workloads_all_variants(scale):
             assert st.rounds == R
 
 
+LDF_VARIANTS = [("maxmin", gcb.MAXMIN, lambda g, s: O.color_maxmin(g, s, ldf=True)),
+                ("luby", gcb.LUBY_MIS, lambda g, s: O.color_luby(g, s, ldf=True)),
+                ("is_alg2", gcb.IS_ALG2, lambda g, s: O.color_is_alg2(g, s, ldf=True)),
+                ("jp_alg4", gcb.JP_ALG4, lambda g, s: O.color_jp_alg4(g, s, ldf=True))]
+
+
+def test_ldf_random_and_workload_graphs():
+    """largest-degree-first priorities (R21) in the COUNT kernels,
+    element by element against the oracle: random graphs, duplicate entries
+    (the degree counts distinct neighbours), a star (closed form), R-MAT s16,
+    ER, the mesh and RGG; max-min rounds and frontier sizes too."""
+    rng = random.Random(12)
+    graphs = [G.random_graph(rng.randint(1, 300), rng.choice([0.02, 0.1, 0.4]), seed=500 + i)
+              for i in range(60)]
+    graphs += [G.rmat(16, 16, seed=2), G.erdos_renyi(30000, 240000, seed=4), G.mesh3d(24, 24, 24),
+               G.rgg(15, seed=1), _csr_tensors(5001, [(0, i) for i in range(1, 5001)])]
+    for i, g in enumerate(graphs):
+        for name, v, ref_fn in LDF_VARIANTS:
+            C, k, st = gpu_colors(g, 1 + i % 5, gcb.LDF(v), frontier_cap=8192)
+            ref = ref_fn(g, 1 + i % 5)
+            assert st.mode_used == gcb.MODE_COUNT
+            assert (C == ref).all(), (name, g.name, i)
+            if name == "maxmin":
+                _, R, nk = O.color_maxmin(g, 1 + i % 5, with_stats=True, ldf=True)
+                assert st.rounds == R and st.frontier_sizes == nk
+    star = graphs[-1]
+    C, _, _ = gpu_colors(star, 3, gcb.LDF(gcb.MAXMIN))
+    assert C[0] == 0 and (C[1:] == 1).all()
+    # duplicates + shuffled rows: same colouring as the clean graph
+    g = G.erdos_renyi(4000, 30000, seed=8)
+    ro, ci = g.row_offsets.tolist(), g.col_indices.tolist()
+    rows = []
+    for v in range(g.n):
+        r = ci[ro[v]:ro[v + 1]]
+        r = r + rng.sample(r, min(len(r), 2))
+        rng.shuffle(r)
+        rows.append(r)
+    nro = [0]
+    for r in rows:
+        nro.append(nro[-1] + len(r))
+    g2 = G.Graph(g.n, torch.tensor(nro, dtype=torch.int64),
+                 torch.tensor([x for r in rows for x in r], dtype=torch.int32))
+    for name, v, ref_fn in LDF_VARIANTS:
+        C, _, _ = gpu_colors(g2, 5, gcb.LDF(v))
+        assert (C == ref_fn(g, 5)).all(), name
+
+
+def test_ldf_rmat_s24_certificates_and_errors():
+    """LDF at the bench size: the max-min certificate and the mex certificate
+    with (degree, weight) keys check every vertex; LDF with multi-hash, Hash IS
+    or a partitioned handle is rejected."""
+    g = G.config_graph("cfg4", device="cuda")
+    gh = g.to("cpu")
+    with gcb.Graph(g.n, g.row_offsets, g.col_indices, flags=gcb.BORROW_DEVICE) as h:
+        out = torch.empty(g.n, dtype=torch.int32, device="cuda")
+        _, k, st = h.color(1, gcb.LDF(gcb.MAXMIN), out, stats=True)
+        C = out.cpu().numpy().view(np.uint32)
+        assert O.cert_maxmin(gh, 1, 1, C, ldf=True) == 0 and O.check_proper(gh, C) == 0
+        assert k in (2 * st.rounds - 1, 2 * st.rounds)
+        _, k, st = h.color(1, gcb.LDF(gcb.LUBY_MIS), out, stats=True)
+        L = out.cpu().numpy().view(np.uint32)
+        assert O.cert_mex(gh, 1, L, ldf=True) == 0 and O.check_proper(gh, L) == 0
+        for bad in (gcb.LDF(gcb.MULTIHASH(2)), gcb.LDF(gcb.HASH_IS(4)), gcb.MAXMIN | (1 << 20)):
+            with pytest.raises(gcb.GCError) as e:
+                h.color(1, bad, out)
+            assert e.value.code == -1
+
+
 def test_cfg5_rmat_s27_one_gpu_and_partitions():
     """cfg5 at its stated size: R-MAT s27 ef16 (1.3e8 vertices, nnz > 2^31).
     One B200 colours it through gc_create_csr / AUTO (the bench launch
