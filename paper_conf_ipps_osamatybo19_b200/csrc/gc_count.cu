@@ -65,6 +65,16 @@ constexpr bool kCountStream = GC_COUNT_STREAM != 0;
                         // (item load, column ids, atomics) in round_stats slots 9, 11-15
 #endif
 
+#ifndef GC_PROF_FRESH
+#define GC_PROF_FRESH 0  // 1 (PROF builds only): end-of-round breakdown (fresh row loads, long-row
+                         // expansion, flush reservation) in round_stats slots 9, 12, 14, 15
+#endif
+
+#ifndef GC_EAGER_RO
+#define GC_EAGER_RO 0  // 1: the lane that frees w loads w's row offsets right away (max-min walk)
+                       // instead of one thread per fresh vertex after the block's units
+#endif
+
 #ifndef GC_PACKED
 #define GC_PACKED 0  // 1: 32-bit (hi << 16 | lo) round counts -- max-min only (no JP / multi-hash branch);
                      // measured 27.9 vs 28.1 ms on R-MAT s24, not worth the restriction
@@ -86,6 +96,7 @@ constexpr int kThreads = GC_COUNT_THREADS;  // one block per SM
 constexpr int kShortMax = 32;              // SL rows: one 8-lane group
 constexpr int kSeg = 256;                  // WL item: one warp, 8 entries per lane
 constexpr int kHubMin = 4096;              // k_count: longer rows by blocks
+constexpr uint32_t kInlineSeg = 4;         // schedule_fresh: rows of <= 4 segments written inline
 constexpr int kHubChunk = 4096;
 constexpr uint32_t kFirst = 0x80000000u;   // item flag: colour v in this round
 constexpr uint32_t kLoSide = 0x40000000u;  // item flag: scheduled by its lo side (min colour)
@@ -129,7 +140,8 @@ enum : int {
     cPhaseNs = 211, // PROF: ns in the init phase, the rounds
     cHubs = 224,    // k_count: hub rows
     cSlot = 240,    // JP: mex slots handed out (monotone)
-    kCCtrWords = 256
+    cRW = 256,      // round words: [16 * (slot * kNG + group)], 3 rotating slots x kNG groups
+    kCCtrWords = 512
 };
 
 struct CArgs {
@@ -231,11 +243,19 @@ __device__ __forceinline__ uint32_t atom_add_global32(uint32_t *p, uint32_t x) {
     return old;
 }
 
-// Round word R (one per round, 3 rotating slots): SL item count in bits
-// [0, 29), WL item count in [29, 53), barrier arrivals in [53, 64).  A block
-// reserves its items of the next round with ONE atomic (both list bases come
-// back), and the spin that ends the round's barrier reads the next round's
-// item counts in the same load that sees the last arrival.
+// Round words (3 rotating slots per group): SL item count in bits [0, 29),
+// WL item count in [29, 53), barrier arrivals in [53, 64).  The blocks are
+// split into kNG groups (block b: group b % kNG), each with its own round
+// words and item arrays, so a word takes ~G / kNG same-address atomics per
+// round instead of G (they serialise in one L2 slice).  A block reserves its
+// items of the next round with ONE atomic on its group's word (both list
+// bases come back); the spin that ends the round's barrier loads every
+// group's word and so reads the next round's item counts in the same loads
+// that see the last arrivals.
+#ifndef GC_BARRIER_GROUPS
+#define GC_BARRIER_GROUPS 1  // measured on R-MAT s24 (persistent kernel): 1 group 23.9 ms, 2: 24.5, 4: 26.0, 8: 29.7
+#endif
+constexpr int kNG = GC_BARRIER_GROUPS;
 constexpr unsigned long long kRwWL = 1ull << 29, kRwArr = 1ull << 53;
 constexpr unsigned long long kMSL = kRwWL - 1ull, kMWL = (1ull << 24) - 1ull;
 __device__ __forceinline__ unsigned long long rw_field(unsigned long long v, int li) {
@@ -245,22 +265,35 @@ __device__ __forceinline__ unsigned long long rw_add(unsigned long long c, int l
     return li == 0 ? c : c << 29;
 }
 
-// Grid barrier on the round word rw (all blocks resident, cooperative
-// launch): release arrival, acquire spin (which also invalidates the SM's
-// L1, so the next phase sees what other SMs wrote); thread 0 leaves the final
-// word in *out.  A wait beyond 4 s records a trap and makes every block leave
+// Grid barrier over the round words of ring slot `slot` (all blocks resident,
+// cooperative launch): release arrival on the block's group word, acquire
+// spin over all groups' words (which also invalidates the SM's L1, so the
+// next phase sees what other SMs wrote); thread 0 leaves the final words in
+// out[0..kNG).  A wait beyond 4 s records a trap and makes every block leave
 // instead of hanging the GPU.
-__device__ __forceinline__ bool grid_barrier_rw(const CArgs &a, uint32_t k, unsigned long long *rw,
+__device__ __forceinline__ unsigned long long *round_word(const CArgs &a, int slot, int grp) {
+    return a.ctr + cRW + 16 * (slot * kNG + grp);
+}
+__device__ __forceinline__ unsigned group_size(int grp) {
+    return (gridDim.x - (unsigned)grp + kNG - 1) / kNG;
+}
+__device__ __forceinline__ bool grid_barrier_rw(const CArgs &a, uint32_t k, int slot,
                                                 unsigned long long *out) {
     __shared__ int ok_sh;
     __syncthreads();
     if (threadIdx.x == 0) {
         int ok = 1;
-        atom_add_release(rw, kRwArr);
+        atom_add_release(round_word(a, slot, (int)(blockIdx.x % kNG)), kRwArr);
         unsigned spins = 0;
         const unsigned long long t0 = gtimer();
-        unsigned long long v;
-        while (((v = ld_acquire(rw)) >> 53) < gridDim.x) {
+        for (;;) {
+            bool done = true;
+#pragma unroll
+            for (int gq = 0; gq < kNG; ++gq) {
+                out[gq] = ld_acquire(round_word(a, slot, gq));
+                done = done && (out[gq] >> 53) >= group_size(gq);
+            }
+            if (done) break;
             if ((++spins & 255u) == 0u) {
                 if (*(volatile unsigned long long *)(a.ctr + cAbort)) {
                     ok = 0;
@@ -274,7 +307,6 @@ __device__ __forceinline__ bool grid_barrier_rw(const CArgs &a, uint32_t k, unsi
                 }
             }
         }
-        *out = v;
         ok_sh = ok;
     }
     __syncthreads();
@@ -299,6 +331,9 @@ struct Stage {
     Item s[kStS];
     Item w[kStW];
     uint2 fresh[kStF];              // (w, lo side?) this block scheduled in the round
+#if GC_EAGER_RO
+    longlong2 fro[kStF];            // their row offsets (loaded by the freeing lane)
+#endif
 #if GC_PACKED
     uint32_t htab[kHTab];           // hash set of the big vertices (kNone = empty)
 #endif
@@ -321,7 +356,10 @@ struct Stage {
     unsigned long long *rw;         // the next round's word R (item reservations, arrivals)
     unsigned long long nbase[2];    // where the next round's items start
     unsigned long long *ccol;       // coloured-count slot of this round
-    unsigned long long rd[4];       // round word from the barrier; SL / WL item counts, trap flag
+    unsigned long long rd[kNG];     // the groups' round words from the barrier
+    unsigned long long gn[2][kNG + 1];  // per list: prefix of the groups' item counts of the round
+    unsigned long long g0[2][kNG];  // per list and group: where the round's items start
+    unsigned long long trap;
 };
 constexpr size_t kStageBytes = sizeof(Stage);
 
@@ -344,6 +382,21 @@ __device__ __forceinline__ int big_slot(uint32_t v) {
     (void)v;
     return -1;
 #endif
+}
+
+// this block's group's item array of list li (offset into SL / WL)
+__device__ __forceinline__ size_t grp_base(const CArgs &a, int li) {
+    return (size_t)(blockIdx.x % kNG) * (size_t)(li == 0 ? a.sl_cap : a.wl_cap);
+}
+// the group and index (into that group's array) of item t of the round's
+// list li (items numbered group by group)
+__device__ __forceinline__ const Item *round_item(const CArgs &a, int li, unsigned long long t) {
+    const Stage &st = stage();
+    int gq = 0;
+#pragma unroll
+    for (int x = 1; x < kNG; ++x) gq += t >= st.gn[li][x] ? 1 : 0;
+    return (li == 0 ? a.SL + (size_t)gq * a.sl_cap : a.WL + (size_t)gq * a.wl_cap) + st.g0[li][gq] +
+           (t - st.gn[li][gq]);
 }
 
 // Whole warp converged: lanes with `pred` append `val` to staged list li;
@@ -371,7 +424,7 @@ __device__ __forceinline__ void stage_append(const CArgs &a, bool pred, const It
         if (spill) {
             const unsigned long long at = st.nbase[li] + gb + __popc(sm & ((1u << lane) - 1u));
             const unsigned long long capg = li == 0 ? a.sl_cap : a.wl_cap;
-            if (at < capg) (li == 0 ? a.SL : a.WL)[at] = val;
+            if (at < capg) (li == 0 ? a.SL + grp_base(a, 0) : a.WL + grp_base(a, 1))[at] = val;
             else flag_error(a, 1, 0, val.v);
         }
     }
@@ -398,6 +451,10 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
         const unsigned c0 = min(st.n[0], (unsigned)kStS), c1 = min(st.n[1], (unsigned)kStW);
         // one reservation for both lists
         const unsigned long long rv = (c0 || c1) ? atom_add_global(st.rw, rw_add(c0, 0) + rw_add(c1, 1)) : 0ull;
+        if (GC_PROF_FRESH && prs) {  // the reservation came back
+            asm volatile("" ::"l"(rv));
+            red_max(prs + 9, gtimer() - t_round);
+        }
         const unsigned long long r0 = rw_field(rv, 0), r1 = rw_field(rv, 1);
         if (r0 + c0 > kMSL || r1 + c1 > kMWL) flag_error(a, 9, 0, 0);  // a round word field overflowed
         st.n[0] = c0;
@@ -416,8 +473,9 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
         st.colored = 0;
     }
     __syncthreads();
-    for (unsigned i = threadIdx.x; i < st.n[0]; i += blockDim.x) a.SL[st.base[0] + i] = st.s[i];
-    for (unsigned i = threadIdx.x; i < st.n[1]; i += blockDim.x) a.WL[st.base[1] + i] = st.w[i];
+    Item *const sl = a.SL + grp_base(a, 0), *const wl = a.WL + grp_base(a, 1);
+    for (unsigned i = threadIdx.x; i < st.n[0]; i += blockDim.x) sl[st.base[0] + i] = st.s[i];
+    for (unsigned i = threadIdx.x; i < st.n[1]; i += blockDim.x) wl[st.base[1] + i] = st.w[i];
     __syncthreads();
     if (threadIdx.x < 2) st.n[threadIdx.x] = 0;
     if (prs && threadIdx.x == 0)
@@ -624,12 +682,22 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint64_t pv, in
     for (int q = 0; q < Q; ++q) {
         ovf[q] = false;
         if (fresh[q]) {
+#if GC_EAGER_RO
+            const longlong2 r = make_longlong2(a.ro[w[q]], a.ro[w[q] + 1]);
+#else
             // its row offsets are loaded at the end of the round: start the
             // HBM -> L2 transfer now
             asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ro + w[q]));
+#endif
             const unsigned pos = atomicAdd(&stage().nf, 1u);
-            if (pos < (unsigned)kStF) stage().fresh[pos] = make_uint2(w[q], hi[q] ? 0u : kLoSide);
-            else ovf[q] = true;
+            if (pos < (unsigned)kStF) {
+                stage().fresh[pos] = make_uint2(w[q], hi[q] ? 0u : kLoSide);
+#if GC_EAGER_RO
+                stage().fro[pos] = r;
+#endif
+            } else {
+                ovf[q] = true;
+            }
         }
     }
 #pragma unroll
@@ -757,7 +825,12 @@ __device__ __forceinline__ void walk_mh(const CArgs &a, uint32_t v, int64_t e, i
         if (fresh[q]) {
             asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ro + w[q]));
             const unsigned pos = atomicAdd(&stage().nf, 1u);
-            if (pos < (unsigned)kStF) stage().fresh[pos] = make_uint2(w[q], 0u);
+            if (pos < (unsigned)kStF) {
+                stage().fresh[pos] = make_uint2(w[q], 0u);
+#if GC_EAGER_RO
+                stage().fro[pos] = make_longlong2(a.ro[w[q]], a.ro[w[q] + 1]);
+#endif
+            }
             else ovf[q] = true;
         }
     }
@@ -808,15 +881,23 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
     if (prs && threadIdx.x == 0) {  // PROF: this block's units are done
         const unsigned long long dt = gtimer() - t_round;
         red_max(prs + 7, dt);
-        if (!GC_PROF_UNIT) red_max(prs + 9, ~dt);  // min via ~
+        if (!GC_PROF_UNIT && !GC_PROF_FRESH) red_max(prs + 9, ~dt);  // min via ~
         if (!GC_PROF_UNIT) red_max(prs + 13, (unsigned long long)st.nf);
         st.t_fs = gtimer();
     }
     const unsigned nf = min(st.nf, (unsigned)kStF);
     for (unsigned t = threadIdx.x; t < nf; t += blockDim.x) {
         const uint2 f = st.fresh[t];
+#if GC_EAGER_RO
+        const int64_t rs = st.fro[t].x, re = st.fro[t].y;
+#else
         const int64_t rs = a.ro[f.x], re = a.ro[f.x + 1];
+#endif
         const int64_t len = re - rs;
+        if (GC_PROF_FRESH && prs) {  // this thread's row offsets are in
+            asm volatile("" ::"l"(len));
+            red_max(prs + 14, gtimer() - t_round);
+        }
         const uint32_t fl = kFirst | f.y;
         if (len <= kShortMax) {
             Item it;
@@ -832,7 +913,7 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
                 st.s[pos] = it;
             } else {
                 const unsigned long long at = st.nbase[0] + rw_field(atom_add_global(st.rw, 1ull), 0);
-                if (at < a.sl_cap) a.SL[at] = it;
+                if (at < a.sl_cap) a.SL[grp_base(a, 0) + at] = it;
                 else flag_error(a, 1, 0, f.x);
             }
         } else {
@@ -847,37 +928,40 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
                 for (unsigned h = sb; h < (unsigned)kStW && h < sb + nseg; ++h) st.w[h].v = kNone;
                 dst = ~(int64_t)(st.nbase[1] + rw_field(atom_add_global(st.rw, rw_add(nseg, 1)), 1));
             }
-            const unsigned li = atomicAdd(&st.nlong, 1u);
+            // rows of <= kInlineSeg segments: this thread writes them now; longer
+            // ones are expanded after the block barrier, one warp per row
+            const unsigned li = nseg <= kInlineSeg ? (unsigned)kLongMax : atomicAdd(&st.nlong, 1u);
             if (li < (unsigned)kLongMax) {
                 st.lng[li].rs = rs;
                 st.lng[li].dst = dst;
                 st.lng[li].w = f.x;
                 st.lng[li].len = (uint32_t)len;
                 st.lng[li].flags = fl;
-            } else {  // long-row list full: this thread writes the segments itself
+            } else {  // short enough, or the long-row list is full: this thread writes them
                 for (uint32_t q = 0; q < nseg; ++q) {
                     Item si;
                     si.v = f.x;
                     si.e0 = rs + (int64_t)q * kSeg;
                     si.lf = (uint32_t)min((int64_t)kSeg, len - (int64_t)q * kSeg) | ((q == 0 || (JP && a.jpv == 1)) ? fl : 0u);
                     if (dst >= 0) st.w[dst + q] = si;
-                    else a.WL[~dst + q] = si;
+                    else a.WL[grp_base(a, 1) + ~dst + q] = si;
                 }
             }
         }
     }
     __syncthreads();
+    if (GC_PROF_FRESH && prs && threadIdx.x == 0) red_max(prs + 15, gtimer() - t_round);
     const unsigned nl = min(st.nlong, (unsigned)kLongMax);
-    for (unsigned r = 0; r < nl; ++r) {
+    for (unsigned r = threadIdx.x >> 5; r < nl; r += blockDim.x >> 5) {  // a warp per long row
         const Stage::Long L = st.lng[r];
         const uint32_t nseg = (L.len + kSeg - 1) / kSeg;
-        for (uint32_t q = threadIdx.x; q < nseg; q += blockDim.x) {
+        for (uint32_t q = lane_id(); q < nseg; q += 32) {
             Item si;
             si.v = L.w;
             si.e0 = L.rs + (int64_t)q * kSeg;
             si.lf = (uint32_t)min((int64_t)kSeg, (int64_t)L.len - (int64_t)q * kSeg) | ((q == 0 || (JP && a.jpv == 1)) ? L.flags : 0u);
             if (L.dst >= 0) st.w[L.dst + q] = si;
-            else a.WL[~L.dst + q] = si;
+            else a.WL[grp_base(a, 1) + ~L.dst + q] = si;
             if (GC_PREFETCH_WL) {  // the segment walked next round: HBM -> L2 now
                 const uint32_t ln = si.lf & kLenMask;
                 for (uint32_t o = 0; o < ln; o += 32) asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ci + si.e0 + o));
@@ -1028,13 +1112,16 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
         // init appends round 0's items to slot 0 at position 0; its colourings
         // count for round 0 (so the "next round" targets are round 0's here)
         if (threadIdx.x == 0) {
-            st.rw = a.ctr + cS;  // round 0's word
+            st.rw = round_word(a, 0, (int)(blockIdx.x % kNG));  // round 0's word
             st.nbase[0] = st.nbase[1] = 0ull;
             st.ccol = a.ctr + cK;
         }
         __syncthreads();
     }
     // ---------------------------------------------------- init = round 0
+    // N_0 = n (written here: a colouring whose round 0 walks no row ends
+    // before the round loop's bookkeeping)
+    if (gtid == 0 && a.nk_cap > 0) a.nk[0] = n;
     // lane per vertex: a zero count colours v in round 0 (min wins, R9)
     for (unsigned long long base = gwarp * 32; base < (unsigned long long)n; base += nwarps * 32) {
         const uint32_t v = (uint32_t)(base + lane);
@@ -1086,7 +1173,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
         schedule_rows<JP>(a, zero && re > rs, v, rs, re - rs, 0u);  // walked in round 0
     }
     stage_flush(a);
-    if (!grid_barrier_rw(a, 0, a.ctr + cS, &stage().rd[0])) return;
+    if (!grid_barrier_rw(a, 0, 0, stage().rd)) return;
     if (PROF && gtid == 0) {
         const unsigned long long t = gtimer();
         a.ctr[cPhaseNs] = t - t0;
@@ -1098,7 +1185,9 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
     const unsigned wpb = blockDim.x >> 5;
     const unsigned long long u_first =
         (unsigned long long)(threadIdx.x >> 5) * gridDim.x + blockIdx.x;
-    unsigned long long sl0 = 0, wl0 = 0;  // where round k's items start
+    unsigned long long sl0[kNG], wl0[kNG];  // per group: where round k's items start
+#pragma unroll
+    for (int gq = 0; gq < kNG; ++gq) sl0[gq] = wl0[gq] = 0;
     int64_t rem = n;                      // gtid 0 only: uncoloured at the round start
     uint32_t last = 0;                    // last round with a colouring
     uint32_t k = 0;
@@ -1112,22 +1201,33 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
         // kernel at most 32 rounds later, grid-uniformly)
         if (threadIdx.x == 0) {
             Stage &st = stage();
-            const unsigned long long w = st.rd[0];
-            const unsigned long long r_ns = rw_field(w, 0), r_nw = rw_field(w, 1);
-            st.rd[1] = r_ns;
-            st.rd[2] = r_nw;
-            st.rd[3] = (k & 31u) == 0u ? __ldcg(&a.ctr[cErr]) : 0ull;
-            st.rw = a.ctr + cS + 16 * (int)((k + 1) % 3);
-            st.nbase[0] = sl0 + r_ns;
-            st.nbase[1] = wl0 + r_nw;
+            const int me = (int)(blockIdx.x % kNG);
+            st.gn[0][0] = st.gn[1][0] = 0;
+#pragma unroll
+            for (int gq = 0; gq < kNG; ++gq) {
+                const unsigned long long r_ns = rw_field(st.rd[gq], 0), r_nw = rw_field(st.rd[gq], 1);
+                st.gn[0][gq + 1] = st.gn[0][gq] + r_ns;
+                st.gn[1][gq + 1] = st.gn[1][gq] + r_nw;
+                st.g0[0][gq] = sl0[gq];
+                st.g0[1][gq] = wl0[gq];
+                if (gq == me) {
+                    st.nbase[0] = sl0[gq] + r_ns;
+                    st.nbase[1] = wl0[gq] + r_nw;
+                }
+            }
+            st.trap = (k & 31u) == 0u ? __ldcg(&a.ctr[cErr]) : 0ull;
+            st.rw = round_word(a, (int)((k + 1) % 3), me);
             st.ccol = a.ctr + cK + 16 * cur;
         }
         __syncthreads();
         if (JP && a.jpv == 3) jp4_round_top(a, k, gtid == 0);
-        const unsigned long long ns = stage().rd[1], nw = stage().rd[2];
-        // word of round k+2 (its last reader: the barrier that ended round k-2)
-        if (gtid == 0) a.ctr[cS + 16 * (int)((k + 2) % 3)] = 0ull;
-        if (stage().rd[3] != 0ull) break;  // a trap fired (uniform: read after a barrier)
+        const unsigned long long ns = stage().gn[0][kNG], nw = stage().gn[1][kNG];
+        // words of round k+2 (their last reader: the barrier that ended round k-2)
+        if (gtid == 0) {
+#pragma unroll
+            for (int gq = 0; gq < kNG; ++gq) *round_word(a, (int)((k + 2) % 3), gq) = 0ull;
+        }
+        if (stage().trap != 0ull) break;  // a trap fired (uniform: read after a barrier)
         if (ns == 0 && nw == 0) break;            // nothing scheduled: done
         if (k >= a.max_rounds) break;
         if (k > 0) last = k;  // every item of round k >= 1 colours (kFirst)
@@ -1135,7 +1235,6 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
             a.rstat[16 * k + 0] = (int64_t)ns;
             a.rstat[16 * k + 1] = (int64_t)nw;
         }
-        const unsigned long long sl1 = sl0 + ns, wl1 = wl0 + nw;
         int64_t *prs = (PROF && (int64_t)k < a.nk_cap) ? a.rstat + 16 * k : nullptr;
         if (prs && threadIdx.x == 0)
             red_max(prs + 6, gtimer() - t_round);
@@ -1147,7 +1246,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
             const long long c_unit = PROF ? clock64() : 0;
             if (u < nw) {
                 // longer rows: one <= kSeg-entry item per warp
-                Item it = a.WL[wl0 + u];
+                Item it = *round_item(a, 1, u);
                 if (it.v == kNone) it.lf = 0;  // hole left by schedule_fresh
                 const uint64_t pv = prio_key(a, it.v);
                 if (JP && a.jpv != 1) {  // Alg.2 / Alg.4: the colour is the round (remapped for Alg.4)
@@ -1194,14 +1293,14 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                 }
             } else if (lane_rows) {
                 // short rows: one per lane, 4 entries per step
-                const unsigned long long idx = sl0 + 32 * (u - nw) + lane;
+                const unsigned long long idx = 32 * (u - nw) + lane;
                 uint32_t v = kNone, len = 0;
                 uint64_t pv = 0;
                 int64_t e0 = 0;
                 bool want = false, cl = false;
                 uint32_t lf = 0, z = 0;
-                if (idx < sl1) {
-                    const Item it = a.SL[idx];
+                if (idx < ns) {
+                    const Item it = *round_item(a, 0, idx);
                     v = it.v;
                     lf = it.lf;
                     len = it.lf & kLenMask;
@@ -1228,14 +1327,14 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                 }
             } else {
                 // short rows: 4 per warp, 8 lanes each, 4 entries per lane
-                const unsigned long long idx = sl0 + 4 * (u - nw) + (lane >> 3);
+                const unsigned long long idx = 4 * (u - nw) + (lane >> 3);
                 uint32_t v = kNone, len = 0;
                 uint64_t pv = 0;
                 int64_t e0 = 0;
                 bool want = false, cl = false;
                 uint32_t lf = 0, z = 0;
-                if (idx < sl1) {
-                    const Item it = a.SL[idx];
+                if (idx < ns) {
+                    const Item it = *round_item(a, 0, idx);
                     v = it.v;
                     lf = it.lf;
                     len = it.lf & kLenMask;
@@ -1265,8 +1364,11 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
             if (prs && lane == 0)
                 red_max(prs + ((GC_PROF_UNIT && u >= nw) ? 13 : 10), (unsigned long long)(clock64() - c_unit));
         }
-        sl0 = sl1;
-        wl0 = wl1;
+#pragma unroll
+        for (int gq = 0; gq < kNG; ++gq) {
+            sl0[gq] += rw_field(stage().rd[gq], 0);
+            wl0[gq] += rw_field(stage().rd[gq], 1);
+        }
         if (PROF) {
             const unsigned s = __reduce_add_sync(kFull, nvis);
             if (lane == 0 && s) atomicAdd(&stage().vis, s);
@@ -1296,7 +1398,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
         }
         schedule_fresh<JP>(a, prs, t_round);
         stage_flush(a, prs, t_round);
-        if (!grid_barrier_rw(a, k, a.ctr + cS + 16 * (int)((k + 1) % 3), &stage().rd[0])) return;
+        if (!grid_barrier_rw(a, k, (int)((k + 1) % 3), stage().rd)) return;
         if (PROF && gtid == 0) {
             const unsigned long long t = gtimer();
             if ((int64_t)k < a.nk_cap) a.rstat[16 * k + 4] = (int64_t)(t - t0);
@@ -1585,7 +1687,11 @@ int launch(gc_graph *g, CArgs &a, int *blocks_out) {
         set_error("persistent count kernel cannot be resident");
         return GC_ERR_CUDA;
     }
-    const int blocks = per_sm * g->sm_count;
+    int blocks = per_sm * g->sm_count;
+    if (const char *eb = std::getenv("GC_COUNT_BLOCKS")) {  // experiments: fewer / more blocks
+        const int b = std::atoi(eb);
+        if (b >= 1 && b <= blocks) blocks = b;
+    }
     if (blocks >= 2048) {  // the round word's arrival field has 11 bits
         set_error("persistent count kernel: too many blocks for the round word");
         return GC_ERR_CUDA;
@@ -1681,8 +1787,9 @@ int ensure_count_scratch(gc_graph *g) {
     GC_CUDA_TRY(dmalloc(&s.Z, nn * 4));
     s.sl_cap = (int64_t)nn;
     s.wl_cap = (int64_t)nn + g->nnz / kSeg + 1;
-    GC_CUDA_TRY(dmalloc(&s.SL, (size_t)s.sl_cap * sizeof(Item)));
-    GC_CUDA_TRY(dmalloc(&s.WL, (size_t)s.wl_cap * sizeof(Item)));
+    // one monotone array per barrier group (each could receive every item)
+    GC_CUDA_TRY(dmalloc(&s.SL, (size_t)kNG * (size_t)s.sl_cap * sizeof(Item)));
+    GC_CUDA_TRY(dmalloc(&s.WL, (size_t)kNG * (size_t)s.wl_cap * sizeof(Item)));
     // hub chunk list: at most nnz / kHubChunk entries
     GC_CUDA_TRY(dmalloc(&s.hubs, ((size_t)g->nnz / kHubChunk + 1) * 8));
     GC_CUDA_TRY(dmalloc(&s.cctr, kCCtrWords * sizeof(unsigned long long)));
