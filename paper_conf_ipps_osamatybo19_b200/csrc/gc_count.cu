@@ -1465,16 +1465,21 @@ __global__ void __launch_bounds__(256) k_count(const int64_t *__restrict__ ro,
             re = ro[v + 1];
         }
         const int64_t deg = re - rs;
-        if (valid && deg <= 16) {
+        // rows of <= 16 entries: one lane each, as many steps as the warp's
+        // longest such row (not always 16: most short rows have 1-4 entries)
+        const bool lrow = valid && deg <= 16;
+        const int dmax = (int)__reduce_max_sync(kFull, lrow ? (unsigned)deg : 0u);
+        if (lrow) {
             uint32_t u[16];
 #pragma unroll
-            for (int q = 0; q < 16; ++q) u[q] = q < deg ? __ldcs(ci + rs + q) : 0u;
+            for (int q = 0; q < 16; ++q) u[q] = (q < dmax && q < deg) ? __ldcs(ci + rs + q) : 0u;
             for (int j = 0; j < H; ++j) {
                 const uint32_t key = keys.k[j];
                 const uint64_t pv = ckey(MH ? nullptr : dg, (uint32_t)v, key);
                 uint32_t h = 0;
 #pragma unroll
-                for (int q = 0; q < 16; ++q) h += (q < deg && ckey(MH ? nullptr : dg, u[q], key) > pv) ? 1u : 0u;
+                for (int q = 0; q < 16; ++q)
+                    if (q < dmax) h += (q < deg && ckey(MH ? nullptr : dg, u[q], key) > pv) ? 1u : 0u;
                 cnt[(size_t)v * H + j] = ((unsigned long long)h << 32) | (unsigned long long)(jp ? 1 : deg - h);
             }
         }
