@@ -569,8 +569,16 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     // rgg (0.63 vs 1.33), R-MAT (26.8 vs 1689) and small grids (64^2: 0.10 vs
     // 0.18, one launch); the plain sweep only on large meshes (128^3: 0.48 vs
     // 0.58; 117^3: 0.43 vs 0.47), whose few uniform rounds stream the CSR.
+    // Large non-skewed graphs: a round's decrements are random 8-byte atomics
+    // over the whole count array, which leaves L2 past ~2^22 vertices; the
+    // sweep's status reads win there (rgg_n_2_23: sweep 7.1 vs count 8.4 ms,
+    // 2^24: 14.3 vs 29.7; 2^22: count 2.2 vs 3.7 -- profiles/r02_rgg_modes.txt).
+    // Skewed graphs (max degree > 8x the mean: power law) take thousands of
+    // rounds and keep COUNT at any size.
+    const bool skewed = g->n > 0 && g->max_deg > 8 * std::max<int64_t>(1, g->nnz / g->n);
     if (mode == GC_MODE_AUTO)
-        mode = (luby || g->max_deg > 8 || g->n < (1 << 20)) ? GC_MODE_COUNT : GC_MODE_SWEEP;
+        mode = (luby || g->n < (1 << 20) || (g->max_deg > 8 && (skewed || g->n <= (1 << 22)))) ? GC_MODE_COUNT
+                                                                                                : GC_MODE_SWEEP;
     if (ldf) mode = GC_MODE_COUNT;  // (degree, weight) keys: COUNT kernels only
     if (luby && mode != GC_MODE_COUNT) mode = GC_MODE_SWEEP;
     if (H != 1 && mode != GC_MODE_COUNT) mode = GC_MODE_SWEEP;  // multi-hash: SWEEP or COUNT
