@@ -336,7 +336,9 @@ def main():
         st.mode_used, str(st.mode_used))
     if use_dist:
         mode_used = {1: "sweep", 4: "count"}.get(st.mode_used, str(st.mode_used)) + \
-            " (1D vertex ranges, per-round NCCL all-gather of coloured pairs)"
+            (" (1D vertex ranges; one persistent kernel per rank, coloured pairs pushed into the peers' "
+             "inboxes over NVLink peer memory each round)" if st.mode_used == 4 else
+             " (1D vertex ranges, per-round NCCL all-gather of coloured pairs)")
 
     # ---- roofline: the COUNT kernels' un-instrumented event times from the
     # timed steps (libgc brackets the counting pass and the persistent kernel

@@ -160,6 +160,8 @@ int dist_exchange(gc_graph *g, size_t bytes, const std::vector<const void *> &se
 void destroy_dist(gc_graph *g) {
     if (!g || !g->dist) return;
     Dist &d = *g->dist;
+    cudaDeviceSynchronize();  // the inboxes may be peer-mapped: no pending work may use them
+    free_inboxes(d);
     for (auto &p : d.parts) free_part(p);
     if (d.host_cnt) hfree(d.host_cnt);
 #ifdef GC_HAVE_NCCL

@@ -45,6 +45,16 @@ struct Part {
     DCState dc;
 };
 
+// Device-driven rounds (gc_dist_count.cu): every partition's
+// inbox -- the coloured pairs the other partitions push to it each round and
+// their per-round mailbox words.  Partition q's inbox lives in q's memory;
+// on one GPU (loopback) all inboxes are local, across GPUs the other ranks'
+// are mapped through CUDA IPC (NVLink peer access).
+struct Inbox {
+    uint2 *recv = nullptr;               // [2 slots][world sources][cap] pairs
+    unsigned long long *mbox = nullptr;  // [2 slots][world sources] words
+};
+
 struct Dist {
     int64_t n_global = 0;
     int world = 1;
@@ -56,10 +66,17 @@ struct Dist {
 #ifdef GC_HAVE_NCCL
     ncclComm_t comm = nullptr;
 #endif
+    // device-driven rounds: inboxes of all partitions (index = partition id)
+    std::vector<Inbox> inbox;
+    std::vector<void *> ipc_opened;      // peer mappings to close (multi-GPU)
+    void *own_recv = nullptr, *own_mbox = nullptr;  // this rank's cudaMalloc'd inbox (multi-GPU)
+    int persist_state = 0;               // 0 not set up, 1 ready, -1 unavailable (host rounds)
+    uint32_t epoch = 0;                  // colourings run (mailbox tags)
 };
 
 
 int run_dist_count(gc_graph *g, const RunParams &p, RunResult *r, int64_t *frontier, int64_t fcap);
+void free_inboxes(Dist &d);
 void free_dist_count(Part &p);
 int dist_reslice(gc_graph *g);  // after gc_dedup.cu replaced the handle's rows
 int dist_exchange(gc_graph *g, size_t bytes, const std::vector<const void *> &send,

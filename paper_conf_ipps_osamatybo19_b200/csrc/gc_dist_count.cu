@@ -20,6 +20,9 @@
 #include <cub/cub.cuh>
 
 #include <algorithm>
+#include <cstdio>
+#include <cstdlib>
+#include <cstring>
 #include <vector>
 
 #include "gc_dist.cuh"
@@ -311,6 +314,371 @@ __global__ void k_dc_long(DCArgs a) {
     if (last_block(a)) dc_advance(a);  // the round is complete on this rank
 }
 
+// ------------------------------------------------ device-driven rounds
+// One persistent cooperative launch per rank runs every round of the
+// partitioned COUNT colouring; no host synchronisation and no
+// per-round launch.  The blocks of the launch are split into one group per
+// local partition (loopback: P partitions on one GPU; across GPUs: one per
+// rank).  Round k of partition p:
+//   A. its scheduled vertices S[lo, hi): colour (2k + lo-free, R9), PUSH the
+//      pair (v, colour) into every other partition's inbox (peer memory
+//      across GPUs: plain stores over NVLink), walk short own rows, queue
+//      long ones;
+//   B. group barrier; the group leader publishes (round tag, pairs, error)
+//      in every other partition's mailbox with a system-scope release;
+//   C. wait for every other partition's mailbox word of round k (acquire):
+//      all pairs of the round are in p's inbox, and every partition now
+//      holds the same totals (the termination / stall decisions agree);
+//   D. apply the received pairs to C and walk their ghost rows, queue long
+//      ones; group barrier; E. long rows and ghost rows by the whole group;
+//      group barrier -- every decrement of round k precedes round k+1.
+// Inbox and mailbox slots alternate with k % 2: a partition writes round
+// k+2's pairs only after it has waited for round k+1's words, which p
+// publishes after its own step D of round k.  Mailbox words carry the
+// colouring epoch, so no clearing (and no host barrier) is needed between
+// colourings.
+constexpr int kMaxLocal = 8;     // local partitions per launch (loopback P <= 8)
+constexpr int64_t kPLongMin = 32;  // rows / ghost rows longer: block chunks (one batch of kQ per thread)
+constexpr int kMaxWorld = 64;
+struct DPArgs {
+    DCArgs part[kMaxLocal];
+    Inbox box[kMaxWorld];
+    int world, nlocal, first;
+    uint32_t epoch;
+    int64_t cap;
+    int64_t n_global;
+    unsigned long long *gbar;    // [kMaxLocal * 16] group barrier counters (monotone per launch)
+    unsigned long long *res;     // [kMaxLocal * 16]: rounds, error, remaining (group leader writes)
+    int64_t *nk;                 // frontier sizes N_k (first local partition)
+    int64_t nk_cap;
+    uint32_t max_rounds;
+    int sys;                     // 1: partitions on other GPUs (system-scope fences), 0: one GPU
+    unsigned long long *tl;      // GC_DIST_TIMELINE: per round 5 maxima (ns since the round top), or null
+    int64_t tl_cap;
+};
+enum : int { cPairs2 = 10, cGChunks2 = 12, cChunks2 = 14 };  // [k % 2] per-round counters (DCState ctr)
+
+__device__ __forceinline__ unsigned long long mbox_word(uint32_t epoch, uint32_t k, unsigned long long cnt,
+                                                        unsigned long long err) {
+    return ((unsigned long long)(epoch & 0xFFFFu) << 48) | ((unsigned long long)((k + 1u) & 0xFFFFu) << 32) |
+           ((err & 3ull) << 30) | (cnt & 0x3FFFFFFFull);
+}
+__device__ __forceinline__ unsigned long long mbox_tag(uint32_t epoch, uint32_t k) {
+    return mbox_word(epoch, k, 0, 0) >> 32;
+}
+__device__ __forceinline__ void st_release_sys(unsigned long long *p, unsigned long long v) {
+    asm volatile("st.release.sys.global.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+__device__ __forceinline__ unsigned long long ld_acquire_sys(const unsigned long long *p) {
+    unsigned long long v;
+    asm volatile("ld.acquire.sys.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+    return v;
+}
+__device__ __forceinline__ void st_relaxed_sys(unsigned long long *p, unsigned long long v) {
+    asm volatile("st.relaxed.sys.global.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+__device__ __forceinline__ unsigned long long ld_relaxed_sys(const unsigned long long *p) {
+    unsigned long long v;
+    asm volatile("ld.relaxed.sys.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+    return v;
+}
+__device__ __forceinline__ unsigned long long ld_acquire_gpu(const unsigned long long *p) {
+    unsigned long long v;
+    asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+    return v;
+}
+__device__ __forceinline__ unsigned long long gtimer_dp() {
+    unsigned long long t;
+    asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+    return t;
+}
+
+// group barrier #epoch_no (monotone counter, release arrival / acquire spin);
+// false after 4 s (the error is then recorded by the caller)
+__device__ __forceinline__ bool group_barrier(unsigned long long *ctr, unsigned gsize, unsigned long long nbar) {
+    __shared__ int ok_sh;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        int ok = 1;
+        asm volatile("red.release.gpu.global.add.u64 [%0], %1;" ::"l"(ctr), "l"(1ull) : "memory");
+        const unsigned long long want = nbar * gsize, t0 = gtimer_dp();
+        unsigned spins = 0;
+        while (ld_acquire_gpu(ctr) < want) {
+            if ((++spins & 255u) == 0u && gtimer_dp() - t0 > 4000000000ull) {
+                ok = 0;
+                break;
+            }
+        }
+        ok_sh = ok;
+    }
+    __syncthreads();
+    return ok_sh != 0;
+}
+
+__device__ __forceinline__ void dec_k(const DCArgs &a, uint32_t pv, uint32_t lw, uint32_t wg, uint32_t k) {
+    const bool hi = pv > weight_mix(wg ^ a.key);
+    const unsigned long long old = atomicAdd(a.cnt + lw, hi ? kDecHi : kDecLo);
+    const uint32_t side = hi ? (uint32_t)(old >> 32) : (uint32_t)old;
+    const uint32_t other = hi ? (uint32_t)old : (uint32_t)(old >> 32);
+    if (side == 1u) {
+        if (other != 0u) push_s(a, lw | (hi ? 0u : kLoF));
+        else if (!hi) a.Z[lw] = k + 1u;
+    } else if (side == 0u) {
+        flag(a, 4, wg);
+    }
+}
+// entries [s, e) of an own row (global ids; remote ones skipped) or a ghost
+// row (owned ids), lanes `sub` of `width`; kQ entries per lane in flight (the
+// atomics of a batch are issued together, not one round trip per entry)
+constexpr int kQ = 4;
+template <bool GHOST>
+__device__ __forceinline__ void walk_entries_k(const DCArgs &a, uint32_t pv, int64_t s, int64_t e, int64_t sub,
+                                               int64_t width, uint32_t k) {
+    for (int64_t i0 = s + sub; i0 < e; i0 += kQ * width) {
+        uint32_t lw[kQ], wg[kQ];
+        bool live[kQ];
+#pragma unroll
+        for (int q = 0; q < kQ; ++q) {
+            const int64_t i = i0 + q * width;
+            live[q] = i < e;
+            if (GHOST) {
+                lw[q] = live[q] ? a.gadj[i] : 0u;
+                wg[q] = a.v0 + lw[q];
+            } else {
+                wg[q] = live[q] ? __ldcs(a.ci + i) : 0u;
+                lw[q] = wg[q] - a.v0;
+                live[q] = live[q] && (int64_t)lw[q] < a.n_loc;
+            }
+        }
+        unsigned long long old[kQ];
+        bool hi[kQ];
+#pragma unroll
+        for (int q = 0; q < kQ; ++q) {
+            hi[q] = pv > weight_mix(wg[q] ^ a.key);
+            old[q] = live[q] ? atomicAdd(a.cnt + lw[q], hi[q] ? kDecHi : kDecLo) : 2ull;
+        }
+#pragma unroll
+        for (int q = 0; q < kQ; ++q) {
+            if (!live[q]) continue;
+            const uint32_t side = hi[q] ? (uint32_t)(old[q] >> 32) : (uint32_t)old[q];
+            const uint32_t other = hi[q] ? (uint32_t)old[q] : (uint32_t)(old[q] >> 32);
+            if (side == 1u) {
+                if (other != 0u) push_s(a, lw[q] | (hi[q] ? 0u : kLoF));
+                else if (!hi[q]) a.Z[lw[q]] = k + 1u;
+            } else if (side == 0u) {
+                flag(a, 4, wg[q]);
+            }
+        }
+    }
+}
+// a self-contained chunk of a long row / ghost row (no job indirection in
+// the round's critical chain): first entry, vertex, length | ghost flag
+struct __align__(16) ChunkItem {
+    int64_t c0;
+    uint32_t v;
+    uint32_t len;  // entries | kGhostBit
+};
+constexpr uint32_t kGhostBit = 0x80000000u;
+__device__ __forceinline__ void push_long_k(const DCArgs &a, int64_t s, int64_t e, uint32_t v, uint32_t ghost,
+                                            int par) {
+    // own rows' chunks at [0, LC_cap), ghost rows' at [LC_cap, 2 LC_cap):
+    // separate lists, so each is complete at its own group barrier
+    const uint32_t nch = (uint32_t)((e - s + kChunk - 1) / kChunk);
+    const unsigned long long b = atomicAdd(a.ctr + (ghost ? cGChunks2 : cChunks2) + par, (unsigned long long)nch);
+    if ((int64_t)(b + nch) > a.LC_cap) {
+        flag(a, 3, v);
+        return;
+    }
+    ChunkItem *lc = reinterpret_cast<ChunkItem *>(a.LC) + (ghost ? a.LC_cap : 0);
+    for (uint32_t c = 0; c < nch; ++c) {
+        const int64_t c0 = s + (int64_t)c * kChunk;
+        lc[b + c] = ChunkItem{c0, v, (uint32_t)min((int64_t)kChunk, e - c0) | (ghost ? kGhostBit : 0u)};
+    }
+}
+// chunks [i0, i1) of the round's list, blocks of the group grid-stride
+__device__ __forceinline__ void walk_chunks(const DCArgs &a, bool ghost, unsigned long long i0,
+                                            unsigned long long i1, unsigned gb, unsigned gsize, uint32_t k) {
+    const ChunkItem *lc = reinterpret_cast<const ChunkItem *>(a.LC) + (ghost ? a.LC_cap : 0);
+    for (unsigned long long i = i0 + gb; i < i1; i += gsize) {
+        const ChunkItem c = lc[i];
+        const uint32_t pv = weight_mix(c.v ^ a.key);
+        const int64_t c1 = c.c0 + (c.len & ~kGhostBit);
+        if (c.len & kGhostBit) walk_entries_k<true>(a, pv, c.c0, c1, threadIdx.x, blockDim.x, k);
+        else walk_entries_k<false>(a, pv, c.c0, c1, threadIdx.x, blockDim.x, k);
+    }
+}
+
+__global__ void __launch_bounds__(256) k_dc_persistent(const __grid_constant__ DPArgs A) {
+    const unsigned gsize = gridDim.x / (unsigned)A.nlocal;
+    const unsigned lp = blockIdx.x / gsize;
+    if (lp >= (unsigned)A.nlocal) return;  // blocks beyond the groups
+    const unsigned gb = blockIdx.x - lp * gsize;
+    const DCArgs &a = A.part[lp];
+    const int p = A.first + (int)lp;
+    const unsigned lane = lane_id();
+    const int64_t gid = ((int64_t)gb * blockDim.x + threadIdx.x) >> 3;  // 8-lane group in the group
+    const int64_t ng = ((int64_t)gsize * blockDim.x) >> 3;
+    const int64_t sub = lane & 7u;
+    unsigned long long *bar = A.gbar + 16 * lp;
+    unsigned long long nbar = 0;
+    __shared__ unsigned long long peer_cnt[kMaxWorld];
+    __shared__ unsigned long long sh_tot, sh_err, sh_nrecv;
+    int64_t remaining = A.n_global;
+    int64_t lo = (int64_t)__ldcg(a.ctr + cLo), hi = (int64_t)__ldcg(a.ctr + cHi);
+    uint32_t k = 0;
+    unsigned long long err_out = 0;
+    for (;; ++k) {
+        const int par = (int)(k & 1u), npar = par ^ 1;
+        const unsigned long long t_round = A.tl ? gtimer_dp() : 0ull;
+        unsigned long long *tl = (A.tl && (int64_t)k < A.tl_cap && threadIdx.x == 0) ? A.tl + 8 * k : nullptr;
+        if (gb == 0 && threadIdx.x == 0) {  // the next round's counters (last used in round k-1)
+            a.ctr[cPairs2 + npar] = 0ull;
+            a.ctr[cGChunks2 + npar] = 0ull;
+            a.ctr[cChunks2 + npar] = 0ull;
+            if (lp == 0 && (int64_t)k < A.nk_cap) A.nk[k] = remaining;
+        }
+        // A. own scheduled vertices
+        for (int64_t i = lo + gid; i < hi; i += ng) {
+            const uint32_t it = a.S[i];
+            const uint32_t lv = it & ~kLoF;
+            const uint32_t vg = a.v0 + lv;
+            const int64_t rs = a.ro[lv], re = a.ro[lv + 1];
+            if (sub == 0) {
+                const bool lo_free = (it & kLoF) || a.Z[lv] <= k;
+                const uint32_t c = 2u * k + (lo_free ? 1u : 0u);
+                a.C[vg] = c;
+                const unsigned long long at = atomicAdd(a.ctr + cPairs2 + par, 1ull);
+                if ((int64_t)at < A.cap) {
+                    for (int q = 0; q < A.world; ++q)
+                        if (q != p) A.box[q].recv[((int64_t)par * A.world + p) * A.cap + (int64_t)at] = make_uint2(vg, c);
+                } else {
+                    flag(a, 2, vg);
+                }
+                if (re - rs > kPLongMin) push_long_k(a, rs, re, vg, 0u, par);
+            }
+            if (re - rs <= kPLongMin) walk_entries_k<false>(a, weight_mix(vg ^ a.key), rs, re, sub, 8, k);
+        }
+        // B. publish
+        if (tl) atomicMax(tl + 0, gtimer_dp() - t_round);  // own walks done
+        if (!group_barrier(bar, gsize, ++nbar)) { err_out = 5; break; }
+        if (tl) atomicMax(tl + 1, gtimer_dp() - t_round);  // group barrier 1
+        // the chunks of own long rows are all queued: walk them while the
+        // other partitions' mailbox words are in flight (E1)
+        const unsigned long long n_own = __ldcg(a.ctr + cChunks2 + par);
+        const unsigned long long own = __ldcg(a.ctr + cPairs2 + par);
+        if (gb == 0 && threadIdx.x == 0 && A.world > 1) {
+            const unsigned long long e = __ldcg(a.ctr + cErr) ? 1ull : 0ull;
+            const unsigned long long w = mbox_word(A.epoch, k, own, e);
+            // one system-scope fence, then the words (release pattern): the
+            // pairs pushed by the whole group (ordered before the group
+            // barrier this thread acquired) are visible before any word
+            if (A.sys) asm volatile("fence.acq_rel.sys;" ::: "memory");
+            else asm volatile("fence.acq_rel.gpu;" ::: "memory");
+            for (int q = 0; q < A.world; ++q)
+                if (q != p) st_relaxed_sys(A.box[q].mbox + (int64_t)par * A.world + p, w);
+        }
+        walk_chunks(a, false, 0, n_own, gb, gsize, k);
+        // C. wait for every other partition's word of round k
+        if (threadIdx.x < 32) {  // warp 0: lane q polls source q's word (all in flight together)
+            const unsigned long long tag = mbox_tag(A.epoch, k), t0 = gtimer_dp();
+            unsigned long long w = 0, c = 0, err = 0;
+            bool done = false;
+            unsigned spins = 0, bad = 0;
+            for (;;) {
+                bool mine = true;
+                for (int q = (int)threadIdx.x; q < A.world; q += 32) {
+                    if (q == p) continue;
+                    w = ld_relaxed_sys(A.box[p].mbox + (int64_t)par * A.world + q);
+                    mine = mine && (w >> 32) == tag;
+                }
+                done = __all_sync(0xFFFFFFFFu, mine);
+                if (done) break;
+                if ((++spins & 255u) == 0u && gtimer_dp() - t0 > 4000000000ull) {
+                    bad = 1;
+                    break;
+                }
+            }
+            if (A.world > 1) {  // acquire pattern
+                if (A.sys) asm volatile("fence.acq_rel.sys;" ::: "memory");
+                else asm volatile("fence.acq_rel.gpu;" ::: "memory");
+            }
+            for (int q = (int)threadIdx.x; q < A.world; q += 32) {
+                if (q == p) {
+                    peer_cnt[q] = 0;
+                    continue;
+                }
+                w = ld_relaxed_sys(A.box[p].mbox + (int64_t)par * A.world + q);
+                peer_cnt[q] = w & 0x3FFFFFFFull;
+                c += peer_cnt[q];
+                err |= (w >> 30) & 3ull;
+            }
+            for (int o = 16; o; o >>= 1) {
+                c += __shfl_xor_sync(0xFFFFFFFFu, c, o);
+                err |= __shfl_xor_sync(0xFFFFFFFFu, err, o);
+            }
+            bad = __reduce_or_sync(0xFFFFFFFFu, bad);
+            if (threadIdx.x == 0) {
+                err |= __ldcg(a.ctr + cErr) ? 1ull : 0ull;
+                sh_tot = own + c;
+                sh_err = bad ? 6ull : (err ? 7ull : 0ull);
+            }
+        }
+        __syncthreads();
+        if (tl) atomicMax(tl + 2, gtimer_dp() - t_round);  // all mailboxes in
+        const unsigned long long tot = sh_tot;
+        if (sh_err) { err_out = sh_err; break; }  // an error on some partition: all stop (uniform)
+        if (tot == 0) { err_out = 8; break; }     // a stall: the adjacency is not symmetric
+        // D. remote pairs: C and ghost rows -- one index space over all
+        // sources (peer_cnt holds the exclusive prefix after the scan below),
+        // so every 8-lane group of the partition works at once
+        if (threadIdx.x == 0) {
+            unsigned long long acc = 0;
+            for (int q = 0; q < A.world; ++q) {
+                const unsigned long long c = peer_cnt[q];
+                peer_cnt[q] = acc;
+                acc += c;
+            }
+            sh_nrecv = acc;  // pairs received
+        }
+        __syncthreads();
+        const int64_t nrecv = (int64_t)sh_nrecv;
+        for (int64_t t = gid; t < nrecv; t += ng) {
+            {
+                int q = 0;
+                while (q + 1 < A.world && (int64_t)peer_cnt[q + 1] <= t) ++q;
+                const uint2 pr = A.box[p].recv[((int64_t)par * A.world + q) * A.cap + (t - (int64_t)peer_cnt[q])];
+                const int64_t gs = a.goff[pr.x], ge = a.goff[(int64_t)pr.x + 1];
+                if (sub == 0) {
+                    a.C[pr.x] = pr.y;
+                    if (ge - gs > kPLongMin) push_long_k(a, gs, ge, pr.x, 1u, par);
+                }
+                if (ge - gs <= kPLongMin) walk_entries_k<true>(a, weight_mix(pr.x ^ a.key), gs, ge, sub, 8, k);
+            }
+        }
+        if (tl) atomicMax(tl + 3, gtimer_dp() - t_round);  // ghost walks done
+        if (!group_barrier(bar, gsize, ++nbar)) { err_out = 5; break; }
+        if (tl) atomicMax(tl + 4, gtimer_dp() - t_round);  // group barrier 2
+        // E2. the chunks of long ghost rows (queued after the own ones)
+        walk_chunks(a, true, 0, __ldcg(a.ctr + cGChunks2 + par), gb, gsize, k);
+        if (tl) atomicMax(tl + 5, gtimer_dp() - t_round);  // long chunks done
+        if (!group_barrier(bar, gsize, ++nbar)) { err_out = 5; break; }
+        if (tl) atomicMax(tl + 6, gtimer_dp() - t_round);  // group barrier 3 (round end)
+        remaining -= (int64_t)tot;
+        lo = hi;
+        hi = (int64_t)__ldcg(a.ctr + cSEnd);
+        if (remaining <= 0) {
+            ++k;
+            break;
+        }
+        if (k + 1 >= A.max_rounds) { err_out = 9; ++k; break; }
+    }
+    if (gb == 0 && threadIdx.x == 0) {
+        A.res[16 * lp + 0] = k;
+        A.res[16 * lp + 1] = err_out;
+        A.res[16 * lp + 2] = (unsigned long long)remaining;
+    }
+}
+
 // ---------------------------------------------------------------- ghost rows
 __global__ void k_dc_gcount(const int64_t *ro, const uint32_t *ci, int64_t nnz, uint32_t v0, int64_t n_loc,
                             unsigned long long *gcnt) {
@@ -375,10 +743,10 @@ int ensure_dc(gc_graph *g, Part &p, int64_t n_global) {
         GC_CUDA_TRY(dmalloc(&s.S, nl * 4));
         // long jobs of one round: own rows and ghost rows longer than kLongMin
         // (each at most nnz / kLongMin); chunk items: at most 2 nnz / kChunk + jobs
-        s.L_cap = 2 * (p.nnz / kLongMin) + 16;
+        s.L_cap = 2 * (p.nnz / std::min(kLongMin, kPLongMin)) + 16;  // own + ghost rows longer than the threshold
         s.LC_cap = 2 * (p.nnz / kChunk) + s.L_cap + 16;
         GC_CUDA_TRY(dmalloc(&s.L, (size_t)s.L_cap * sizeof(LongJob)));
-        GC_CUDA_TRY(dmalloc(&s.LC, (size_t)s.LC_cap * sizeof(uint2)));
+        GC_CUDA_TRY(dmalloc(&s.LC, (size_t)s.LC_cap * 32));  // uint2 items (host rounds) or 2 lists of 16 B ChunkItems
         GC_CUDA_TRY(dmalloc(&s.ctr, kDCtrWords * sizeof(unsigned long long)));
     }
     if (!s.ghost_built) return build_ghost(g, p, n_global);
@@ -422,6 +790,217 @@ void free_dist_count(Part &p) {
     dfree(s.gadj);
     dfree(s.ctr);
     s = DCState();
+}
+
+
+// ------------------------------------------------ device-driven rounds: host
+namespace {
+
+// Inboxes of every partition.  One GPU (loopback): device allocations.  Across
+// GPUs: each rank cudaMallocs its inbox, the IPC handles are all-gathered over
+// the rank's NCCL communicator and the peers' inboxes are opened (NVLink peer
+// access); any failure leaves the handle on the host-driven rounds.
+int ensure_inboxes(gc_graph *g) {
+    Dist &d = *g->dist;
+    if (d.persist_state != 0) return GC_OK;
+    const size_t recv_bytes = sizeof(uint2) * 2 * (size_t)d.world * (size_t)std::max<int64_t>(d.cap, 1);
+    const size_t mbox_bytes = sizeof(unsigned long long) * 2 * (size_t)d.world;
+    d.inbox.assign((size_t)d.world, Inbox());
+    if (d.loopback) {
+        for (int q = 0; q < d.world; ++q) {
+            GC_CUDA_TRY(dmalloc(&d.inbox[q].recv, recv_bytes));
+            GC_CUDA_TRY(dmalloc(&d.inbox[q].mbox, mbox_bytes));
+            GC_CUDA_TRY(cudaMemsetAsync(d.inbox[q].mbox, 0, mbox_bytes, g->stream));
+        }
+        d.persist_state = 1;
+        return GC_OK;
+    }
+#ifdef GC_HAVE_NCCL
+    d.persist_state = -1;  // until every step below succeeded
+    if (cudaMalloc(&d.own_recv, recv_bytes) != cudaSuccess || cudaMalloc(&d.own_mbox, mbox_bytes) != cudaSuccess) {
+        cudaGetLastError();
+        return GC_OK;
+    }
+    GC_CUDA_TRY(cudaMemsetAsync(d.own_mbox, 0, mbox_bytes, g->stream));
+    cudaIpcMemHandle_t mine[2];
+    if (cudaIpcGetMemHandle(&mine[0], d.own_recv) != cudaSuccess ||
+        cudaIpcGetMemHandle(&mine[1], d.own_mbox) != cudaSuccess) {
+        cudaGetLastError();
+        return GC_OK;
+    }
+    char *dev = nullptr;
+    const size_t hb = sizeof(mine);
+    GC_CUDA_TRY(dmalloc(&dev, hb * (size_t)(d.world + 1)));
+    GC_CUDA_TRY(cudaMemcpyAsync(dev + hb * (size_t)d.world, mine, hb, cudaMemcpyHostToDevice, g->stream));
+    ncclResult_t ne = ncclAllGather(dev + hb * (size_t)d.world, dev, hb, ncclUint8, d.comm, g->stream);
+    if (ne != ncclSuccess) {
+        dfree(dev);
+        return nccl_fail(ne, "ncclAllGather (inbox handles)");
+    }
+    std::vector<cudaIpcMemHandle_t> all(2 * (size_t)d.world);
+    GC_CUDA_TRY(cudaMemcpyAsync(all.data(), dev, hb * (size_t)d.world, cudaMemcpyDeviceToHost, g->stream));
+    GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
+    dfree(dev);
+    bool ok = true;
+    for (int q = 0; q < d.world && ok; ++q) {
+        if (q == d.rank) {
+            d.inbox[q].recv = reinterpret_cast<uint2 *>(d.own_recv);
+            d.inbox[q].mbox = reinterpret_cast<unsigned long long *>(d.own_mbox);
+            continue;
+        }
+        void *pr = nullptr, *pm = nullptr;
+        if (cudaIpcOpenMemHandle(&pr, all[2 * q], cudaIpcMemLazyEnablePeerAccess) != cudaSuccess) ok = false;
+        else d.ipc_opened.push_back(pr);
+        if (ok && cudaIpcOpenMemHandle(&pm, all[2 * q + 1], cudaIpcMemLazyEnablePeerAccess) != cudaSuccess) ok = false;
+        else if (ok) d.ipc_opened.push_back(pm);
+        d.inbox[q].recv = reinterpret_cast<uint2 *>(pr);
+        d.inbox[q].mbox = reinterpret_cast<unsigned long long *>(pm);
+    }
+    cudaGetLastError();
+    // every rank must agree (a rank without peer access makes all use host rounds)
+    int *flag_d = nullptr;
+    int flag_h = ok ? 1 : 0;
+    GC_CUDA_TRY(dmalloc(&flag_d, sizeof(int)));
+    GC_CUDA_TRY(cudaMemcpyAsync(flag_d, &flag_h, sizeof(int), cudaMemcpyHostToDevice, g->stream));
+    ne = ncclAllReduce(flag_d, flag_d, 1, ncclInt32, ncclMin, d.comm, g->stream);
+    if (ne == ncclSuccess) GC_CUDA_TRY(cudaMemcpyAsync(&flag_h, flag_d, sizeof(int), cudaMemcpyDeviceToHost, g->stream));
+    GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
+    dfree(flag_d);
+    if (ne != ncclSuccess) return nccl_fail(ne, "ncclAllReduce (peer access)");
+    d.persist_state = flag_h ? 1 : -1;
+    return GC_OK;
+#else
+    d.persist_state = -1;
+    return GC_OK;
+#endif
+}
+
+bool use_persistent(gc_graph *g) {
+    Dist &d = *g->dist;
+    const char *e = std::getenv("GC_DIST_HOST_ROUNDS");  // A/B: the host-driven rounds
+    if (e && e[0] == '1') return false;
+    if ((int)d.parts.size() > kMaxLocal || d.world > kMaxWorld) return false;
+    if (ensure_inboxes(g) != GC_OK) return false;
+    return d.persist_state == 1;
+}
+
+int run_dist_persistent(gc_graph *g, const RunParams &p, RunResult *r, int64_t *frontier, int64_t fcap) {
+    Dist &d = *g->dist;
+    cudaStream_t st = g->stream;
+    const int nlocal = (int)d.parts.size();
+    DPArgs A;
+    memset(&A, 0, sizeof(A));
+    for (int lp = 0; lp < nlocal; ++lp) A.part[lp] = args_of(g, d.parts[lp], p.keys.k[0], 0);
+    for (int q = 0; q < d.world; ++q) A.box[q] = d.inbox[q];
+    A.world = d.world;
+    A.nlocal = nlocal;
+    A.first = d.loopback ? 0 : d.rank;
+    A.epoch = ++d.epoch;
+    A.cap = std::max<int64_t>(d.cap, 1);
+    A.n_global = d.n_global;
+    A.max_rounds = (uint32_t)std::min<int64_t>(p.max_rounds, 0xFFFFFFF0ll);
+    A.sys = d.loopback ? 0 : 1;
+    const char *tle = std::getenv("GC_DIST_TIMELINE");  // experiments: per-round phase timeline
+    unsigned long long *tlbuf = nullptr;
+    const int64_t tl_cap = tle ? 1 << 14 : 0;
+    if (tl_cap) {
+        GC_CUDA_TRY(dmalloc(&tlbuf, (size_t)tl_cap * 64));
+        GC_CUDA_TRY(cudaMemsetAsync(tlbuf, 0, (size_t)tl_cap * 64, st));
+    }
+    A.tl = tlbuf;
+    A.tl_cap = tl_cap;
+    const int64_t nk_cap = std::min<int64_t>(fcap > 0 ? fcap : 0, 1 << 20);
+    unsigned long long *scratch = nullptr;  // gbar [16 kMaxLocal] + res [16 kMaxLocal] + nk
+    const size_t words = 32 * (size_t)kMaxLocal + (size_t)std::max<int64_t>(nk_cap, 1);
+    GC_CUDA_TRY(dmalloc(&scratch, words * 8));
+    GC_CUDA_TRY(cudaMemsetAsync(scratch, 0, 32 * (size_t)kMaxLocal * 8, st));
+    A.gbar = scratch;
+    A.res = scratch + 16 * kMaxLocal;
+    A.nk = reinterpret_cast<int64_t *>(scratch + 32 * kMaxLocal);
+    A.nk_cap = nk_cap;
+    int per_sm = 0;
+    GC_CUDA_TRY(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_dc_persistent, 256, 0));
+    const int gsize = std::max(1, (std::min(per_sm, 2) * g->sm_count) / nlocal);
+    cudaLaunchAttribute attr;
+    attr.id = cudaLaunchAttributeCooperative;
+    attr.val.cooperative = 1;
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = dim3((unsigned)(gsize * nlocal));
+    cfg.blockDim = dim3(256);
+    cfg.stream = st;
+    cfg.attrs = &attr;
+    cfg.numAttrs = 1;
+    cudaError_t le = cudaLaunchKernelEx(&cfg, k_dc_persistent, A);
+    if (le != cudaSuccess) {
+        dfree(scratch);
+        return cuda_fail(le, "k_dc_persistent launch");
+    }
+    r->launches += 1;
+    unsigned long long res[16 * kMaxLocal];
+    GC_CUDA_TRY(cudaMemcpyAsync(res, A.res, sizeof(res), cudaMemcpyDeviceToHost, st));
+    std::vector<int64_t> nk((size_t)std::max<int64_t>(nk_cap, 1));
+    if (nk_cap > 0) GC_CUDA_TRY(cudaMemcpyAsync(nk.data(), A.nk, 8 * (size_t)nk_cap, cudaMemcpyDeviceToHost, st));
+    GC_CUDA_TRY(cudaStreamSynchronize(st));
+    dfree(scratch);
+    if (tl_cap) {  // mean over rounds 10.. of each phase end (us), to stderr
+        std::vector<unsigned long long> t((size_t)tl_cap * 8);
+        GC_CUDA_TRY(cudaMemcpy(t.data(), tlbuf, t.size() * 8, cudaMemcpyDeviceToHost));
+        dfree(tlbuf);
+        const int64_t R = std::min<int64_t>((int64_t)res[0], tl_cap);
+        double sum[7] = {0};
+        for (int64_t k = std::min<int64_t>(10, R); k < R; ++k)
+            for (int c = 0; c < 7; ++c) sum[c] += (double)t[8 * k + c];
+        const double cnt = (double)std::max<int64_t>(1, R - std::min<int64_t>(10, R));
+        fprintf(stderr, "dist timeline (us, mean of rounds >= 10, max over blocks): own-walks %.2f bar1 %.2f mbox %.2f "
+                "ghost %.2f bar2 %.2f long %.2f bar3 %.2f\n", sum[0] / cnt / 1e3, sum[1] / cnt / 1e3, sum[2] / cnt / 1e3,
+                sum[3] / cnt / 1e3, sum[4] / cnt / 1e3, sum[5] / cnt / 1e3, sum[6] / cnt / 1e3);
+    }
+    unsigned long long err = 0, local_kind = 0;
+    for (int lp = 0; lp < nlocal; ++lp) {
+        err = std::max(err, res[16 * lp + 1]);
+        unsigned long long c[kDCtrWords];
+        GC_CUDA_TRY(cudaMemcpy(c, d.parts[lp].dc.ctr, sizeof(c), cudaMemcpyDeviceToHost));
+        if (c[cErr]) local_kind = c[cErr];
+    }
+    if (err) {
+        if (err == 5 || err == 6) {
+            set_error("distributed COUNT rounds: a partition stopped answering (device-side timeout)");
+            return d.loopback ? GC_ERR_CUDA : GC_ERR_NCCL;
+        }
+        if (err == 9) {
+            set_error("distributed colouring exceeded the round limit");
+            return GC_ERR_TOO_LARGE;
+        }
+        if (local_kind == 2 || local_kind == 3) {
+            set_error("internal: distributed COUNT list overflow");
+            return GC_ERR_CUDA;
+        }
+        set_error("distributed COUNT colouring: the adjacency is not symmetric");
+        return GC_ERR_NOT_SYMMETRIC;
+    }
+    r->rounds = (int64_t)res[0];
+    r->inner = r->rounds;
+    for (int64_t k = 0; frontier && k < std::min<int64_t>(fcap, r->rounds) && k < nk_cap; ++k) frontier[k] = nk[k];
+    return GC_OK;
+}
+
+}  // namespace
+
+void free_inboxes(Dist &d) {
+    if (d.loopback) {
+        for (auto &b : d.inbox) {
+            dfree(b.recv);
+            dfree(b.mbox);
+        }
+    } else {
+        for (void *ptr : d.ipc_opened) cudaIpcCloseMemHandle(ptr);
+        if (d.own_recv) cudaFree(d.own_recv);
+        if (d.own_mbox) cudaFree(d.own_mbox);
+    }
+    d.inbox.clear();
+    d.ipc_opened.clear();
+    d.own_recv = d.own_mbox = nullptr;
+    d.persist_state = 0;
 }
 
 int run_dist_count(gc_graph *g, const RunParams &p, RunResult *r, int64_t *frontier, int64_t fcap) {
@@ -470,6 +1049,22 @@ int run_dist_count(gc_graph *g, const RunParams &p, RunResult *r, int64_t *front
         r->launches += 4;
     }
     GC_CUDA_TRY(cudaGetLastError());
+    if (use_persistent(g)) {
+        int rc = run_dist_persistent(g, p, r, frontier, fcap);
+        if (rc) return rc;
+        if (prof) {
+            GC_CUDA_TRY(cudaEventRecord(pe1, st));
+            GC_CUDA_TRY(cudaEventSynchronize(pe1));
+            float ms = 0.f;
+            cudaEventElapsedTime(&ms, pe0, pe1);
+            cudaEventDestroy(pe0);
+            cudaEventDestroy(pe1);
+            p.prof->ms[0] += ms;
+            p.prof->launches[0] += 1;
+            p.prof->launch_us.push_back(1e3f * ms);
+        }
+        return GC_OK;
+    }
     std::vector<const void *> cs(d.parts.size()), ps(d.parts.size());
     std::vector<void *> cr(d.parts.size()), pr(d.parts.size());
     for (size_t q = 0; q < d.parts.size(); ++q) {
