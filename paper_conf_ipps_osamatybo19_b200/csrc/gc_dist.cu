@@ -20,6 +20,9 @@
 // colours (no final gather needed).
 #include <algorithm>
 #include <cstring>
+#include <chrono>
+#include <cstdlib>
+#include <thread>
 #include <vector>
 
 #include "gc_dist.cuh"
@@ -27,6 +30,43 @@
 namespace gc {
 
 int fill_u32(uint32_t *p, uint32_t val, int64_t n, cudaStream_t st);
+
+// Wait for the handle's stream after NCCL work: polls the stream and the
+// communicator's asynchronous error state; an NCCL error, or no progress for
+// GC_NCCL_TIMEOUT_S seconds (default 120: a dead or hung peer), aborts the
+// communicator (ncclCommAbort) and returns GC_ERR_NCCL instead of blocking
+// forever in cudaStreamSynchronize.  The handle is unusable after an abort.
+int dist_wait(gc_graph *g) {
+    Dist &d = *g->dist;
+#ifdef GC_HAVE_NCCL
+    if (!d.loopback && d.comm) {
+        double limit = 120.0;
+        if (const char *e = std::getenv("GC_NCCL_TIMEOUT_S")) limit = std::max(1.0, std::atof(e));
+        const auto t0 = std::chrono::steady_clock::now();
+        for (unsigned spins = 0;; ++spins) {
+            const cudaError_t q = cudaStreamQuery(g->stream);
+            if (q == cudaSuccess) return GC_OK;
+            if (q != cudaErrorNotReady) return cuda_fail(q, "distributed round");
+            ncclResult_t ae = ncclSuccess;
+            if (ncclCommGetAsyncError(d.comm, &ae) != ncclSuccess || ae != ncclSuccess) {
+                ncclCommAbort(d.comm);
+                d.comm = nullptr;
+                return nccl_fail(ae, "asynchronous NCCL error (communicator aborted)");
+            }
+            if (std::chrono::duration<double>(std::chrono::steady_clock::now() - t0).count() > limit) {
+                ncclCommAbort(d.comm);
+                d.comm = nullptr;
+                set_error("distributed round: no progress within GC_NCCL_TIMEOUT_S (peer dead or hung); "
+                          "NCCL communicator aborted");
+                return GC_ERR_NCCL;
+            }
+            if (spins > 64) std::this_thread::sleep_for(std::chrono::microseconds(20));
+        }
+    }
+#endif
+    GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
+    return GC_OK;
+}
 
 int nccl_fail(int e, const char *what) {
 #ifdef GC_HAVE_NCCL
@@ -226,7 +266,7 @@ int run_dist(gc_graph *g, const RunParams &p, RunResult *r, int64_t *frontier, i
         GC_CUDA_TRY(cudaMemcpyAsync(d.host_cnt, d.parts[0].cnt_recv,
                                     2 * sizeof(unsigned long long) * d.world,
                                     cudaMemcpyDeviceToHost, g->stream));
-        GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
+        if ((rc = dist_wait(g))) return rc;
         unsigned long long maxc = 0, rem = 0;
         for (int q = 0; q < d.world; ++q) {
             maxc = std::max(maxc, d.host_cnt[2 * q]);

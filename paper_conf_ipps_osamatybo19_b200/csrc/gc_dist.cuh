@@ -82,5 +82,6 @@ int dist_reslice(gc_graph *g);  // after gc_dedup.cu replaced the handle's rows
 int dist_exchange(gc_graph *g, size_t bytes, const std::vector<const void *> &send,
                   const std::vector<void *> &recv);
 int nccl_fail(int e, const char *what);
+int dist_wait(gc_graph *g);  // stream wait with NCCL async-error polling, timeout and abort
 
 }  // namespace gc

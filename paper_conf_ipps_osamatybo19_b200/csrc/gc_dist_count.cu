@@ -839,7 +839,10 @@ int ensure_inboxes(gc_graph *g) {
     }
     std::vector<cudaIpcMemHandle_t> all(2 * (size_t)d.world);
     GC_CUDA_TRY(cudaMemcpyAsync(all.data(), dev, hb * (size_t)d.world, cudaMemcpyDeviceToHost, g->stream));
-    GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
+    if (int rw = dist_wait(g)) {
+        dfree(dev);
+        return rw;
+    }
     dfree(dev);
     bool ok = true;
     for (int q = 0; q < d.world && ok; ++q) {
@@ -864,7 +867,10 @@ int ensure_inboxes(gc_graph *g) {
     GC_CUDA_TRY(cudaMemcpyAsync(flag_d, &flag_h, sizeof(int), cudaMemcpyHostToDevice, g->stream));
     ne = ncclAllReduce(flag_d, flag_d, 1, ncclInt32, ncclMin, d.comm, g->stream);
     if (ne == ncclSuccess) GC_CUDA_TRY(cudaMemcpyAsync(&flag_h, flag_d, sizeof(int), cudaMemcpyDeviceToHost, g->stream));
-    GC_CUDA_TRY(cudaStreamSynchronize(g->stream));
+    if (int rw = dist_wait(g)) {
+        dfree(flag_d);
+        return rw;
+    }
     dfree(flag_d);
     if (ne != ncclSuccess) return nccl_fail(ne, "ncclAllReduce (peer access)");
     d.persist_state = flag_h ? 1 : -1;
@@ -1089,7 +1095,7 @@ int run_dist_count(gc_graph *g, const RunParams &p, RunResult *r, int64_t *front
         if (rc) return rc;
         GC_CUDA_TRY(cudaMemcpyAsync(d.host_cnt, d.parts[0].cnt_recv, 2 * sizeof(unsigned long long) * d.world,
                                     cudaMemcpyDeviceToHost, st));
-        GC_CUDA_TRY(cudaStreamSynchronize(st));
+        if ((rc = dist_wait(g))) return rc;
         unsigned long long maxc = 0, tot = 0, err = 0;
         for (int q = 0; q < d.world; ++q) {
             maxc = std::max(maxc, d.host_cnt[2 * q]);
