@@ -93,8 +93,14 @@ constexpr uint32_t kNever = 0xFFFFFFFFu;  // Z: side never free (yet)
 #define GC_COUNT_THREADS 512
 #endif
 constexpr int kThreads = GC_COUNT_THREADS;  // one block per SM
-constexpr int kShortMax = 32;              // SL rows: one 8-lane group
-constexpr int kSeg = 256;                  // WL item: one warp, 8 entries per lane
+#ifndef GC_SHORT_MAX
+#define GC_SHORT_MAX 32
+#endif
+#ifndef GC_SEG
+#define GC_SEG 128  // measured on R-MAT s24: 128 -> 23.76 ms, 256 -> 23.90, 512 -> 28.4 (GC_SHORT_MAX 16: 24.1)
+#endif
+constexpr int kShortMax = GC_SHORT_MAX;    // SL rows: one 8-lane group
+constexpr int kSeg = GC_SEG;               // WL item: one warp, kSeg / 32 entries per lane
 constexpr int kHubMin = 4096;              // k_count: longer rows by blocks
 constexpr uint32_t kInlineSeg = 4;         // schedule_fresh: rows of <= 4 segments written inline
 constexpr int kHubChunk = 4096;
