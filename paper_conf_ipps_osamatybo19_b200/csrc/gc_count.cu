@@ -262,6 +262,14 @@ __device__ __forceinline__ uint32_t atom_add_global32(uint32_t *p, uint32_t x) {
 #define GC_BARRIER_GROUPS 1  // measured on R-MAT s24 (persistent kernel): 1 group 23.9 ms, 2: 24.5, 4: 26.0, 8: 29.7
 #endif
 constexpr int kNG = GC_BARRIER_GROUPS;
+#ifndef GC_BARRIER_RELAXED_SPIN
+#define GC_BARRIER_RELAXED_SPIN 1
+#endif
+__device__ __forceinline__ unsigned long long ld_relaxed_u64(const unsigned long long *p) {
+    unsigned long long v;
+    asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+    return v;
+}
 constexpr unsigned long long kRwWL = 1ull << 29, kRwArr = 1ull << 53;
 constexpr unsigned long long kMSL = kRwWL - 1ull, kMWL = (1ull << 24) - 1ull;
 __device__ __forceinline__ unsigned long long rw_field(unsigned long long v, int li) {
@@ -289,17 +297,33 @@ __device__ __forceinline__ bool grid_barrier_rw(const CArgs &a, uint32_t k, int 
     __syncthreads();
     if (threadIdx.x == 0) {
         int ok = 1;
+#if GC_BARRIER_RELAXED_SPIN
+        // arrival without a return value (release pattern), relaxed spin,
+        // one acquire fence after the last arrival is seen
+        asm volatile("red.release.gpu.global.add.u64 [%0], %1;" ::"l"(round_word(a, slot, (int)(blockIdx.x % kNG))),
+                     "l"(kRwArr) : "memory");
+#else
         atom_add_release(round_word(a, slot, (int)(blockIdx.x % kNG)), kRwArr);
+#endif
         unsigned spins = 0;
         const unsigned long long t0 = gtimer();
         for (;;) {
             bool done = true;
 #pragma unroll
             for (int gq = 0; gq < kNG; ++gq) {
+#if GC_BARRIER_RELAXED_SPIN
+                out[gq] = ld_relaxed_u64(round_word(a, slot, gq));
+#else
                 out[gq] = ld_acquire(round_word(a, slot, gq));
+#endif
                 done = done && (out[gq] >> 53) >= group_size(gq);
             }
-            if (done) break;
+            if (done) {
+#if GC_BARRIER_RELAXED_SPIN
+                asm volatile("fence.acq_rel.gpu;" ::: "memory");
+#endif
+                break;
+            }
             if ((++spins & 255u) == 0u) {
                 if (*(volatile unsigned long long *)(a.ctr + cAbort)) {
                     ok = 0;
