@@ -173,3 +173,138 @@ def test_partitioned_count_protocol_world2(scale, seed):
         assert p.exitcode == 0
     assert all(r[1] for r in res), "replicated colours differ from the oracle"
     assert all(r[2] for r in res), "round count differs from the oracle"
+
+
+# model of the DEVICE-DRIVEN rounds' exchange (gc_dist_count.cu
+# k_dc_persistent), world size 2 on the CPU: every rank pushes
+# its coloured pairs into the other rank's inbox (shared memory standing in
+# for NVLink peer memory), then writes its mailbox word (epoch | round tag |
+# count) there, and polls its own mailbox for the other rank's word.  Inbox
+# and mailbox slots alternate with the round's parity; two colourings run
+# back to back without clearing anything (the epoch in the word separates
+# them); random delays make the ranks drift apart.  Checked against the
+# oracle: the colouring, and that both ranks took the same decisions.
+def _mailbox_worker(rank, world, port, q, recv, mbox, scale, seeds):
+    import random
+    import time
+
+    import numpy as np
+
+    import oracle as O
+    os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    rng = random.Random(rank * 7 + 1)
+    cap = recv.shape[-1]
+    out = []
+    try:
+        g = G.rmat(scale, 8, seed=3)
+        n = g.n
+        v0, v1 = gdist.split_range(n, world, rank)
+        ro, ci = (t.numpy() for t in gdist.local_rows(g, v0, v1))
+        dist.barrier()  # the inboxes exist on every rank (the IPC handle exchange)
+        for epoch, seed in enumerate(seeds, start=1):
+            p = O.priorities(seed, 0, n).astype(np.int64)
+            nl = v1 - v0
+            hi = np.zeros(nl, dtype=np.int64)
+            lo = np.zeros(nl, dtype=np.int64)
+            ghost = {}
+            for lv in range(nl):
+                row = ci[ro[lv]:ro[lv + 1]].astype(np.int64)
+                hi[lv] = int((p[row] > p[v0 + lv]).sum())
+                lo[lv] = len(row) - hi[lv]
+                for u in row:
+                    if not v0 <= u < v1:
+                        ghost.setdefault(int(u), []).append(lv)
+            UNC, NEVER = 0xFFFFFFFF, 1 << 62
+            C = np.full(n, UNC, dtype=np.uint32)
+            Z = np.full(nl, NEVER, dtype=np.int64)
+            S = [(lv, lo[lv] == 0) for lv in range(nl) if hi[lv] == 0 or lo[lv] == 0]
+            k, remaining, totals = 0, n, []
+            while remaining > 0:
+                par = k & 1
+                nxt = []
+
+                def dec(pv, lw):
+                    if pv > p[v0 + lw]:
+                        hi[lw] -= 1
+                        side, other, lo_side = hi[lw], lo[lw], False
+                    else:
+                        lo[lw] -= 1
+                        side, other, lo_side = lo[lw], hi[lw], True
+                    assert side >= 0
+                    if side == 0:
+                        if other > 0:
+                            nxt.append((lw, lo_side))
+                        elif lo_side:
+                            Z[lw] = k + 1
+                # A: colour the scheduled vertices, push the pairs into the peer's inbox
+                npush = 0
+                for lv, lof in S:
+                    c = 2 * k + (1 if (lof or Z[lv] <= k) else 0)
+                    C[v0 + lv] = c
+                    for qq in range(world):
+                        if qq != rank:
+                            recv[qq, par, rank, npush] = ((v0 + lv) << 32) | c
+                    npush += 1
+                    for u in ci[ro[lv]:ro[lv + 1]]:
+                        if v0 <= u < v1:
+                            dec(p[v0 + lv], int(u) - v0)
+                assert npush <= cap
+                if rng.random() < 0.5:
+                    time.sleep(rng.random() * 0.002)
+                # B: the mailbox words (after the pairs)
+                word = (epoch << 48) | (((k + 1) & 0xFFFF) << 32) | npush
+                for qq in range(world):
+                    if qq != rank:
+                        mbox[qq, par, rank] = word
+                # C: wait for every other rank's word of this round and epoch
+                tot = npush
+                got = {}
+                for qq in range(world):
+                    if qq == rank:
+                        continue
+                    t0 = time.time()
+                    while (int(mbox[rank, par, qq]) >> 32) != ((epoch << 16) | ((k + 1) & 0xFFFF)):
+                        assert time.time() - t0 < 60, "mailbox wait timed out"
+                    got[qq] = int(mbox[rank, par, qq]) & 0x3FFFFFFF
+                    tot += got[qq]
+                assert tot > 0, "stall"
+                # D: the received pairs -> colours and ghost rows
+                for qq, cnt in got.items():
+                    for i in range(cnt):
+                        x = int(recv[rank, par, qq, i])
+                        v, c = x >> 32, x & 0xFFFFFFFF
+                        C[v] = c
+                        for lw in ghost.get(v, ()):
+                            dec(p[v], lw)
+                totals.append(tot)
+                remaining -= tot
+                S = nxt
+                k += 1
+            ref, R, _ = O.color_maxmin(g, seed, with_stats=True)
+            out.append((bool((C == ref).all()), k == R, totals))
+        q.put((rank, out))
+    finally:
+        dist.destroy_process_group()
+
+
+def test_device_driven_mailbox_protocol_world2():
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _free_port()
+    world, scale = 2, 9
+    cap = (1 << scale) // world + 1
+    recv = torch.zeros((world, 2, world, cap), dtype=torch.int64).share_memory_()
+    mbox = torch.zeros((world, 2, world), dtype=torch.int64).share_memory_()
+    procs = [ctx.Process(target=_mailbox_worker, args=(r, world, port, q, recv, mbox, scale, (3, 11)))
+             for r in range(world)]
+    for p in procs:
+        p.start()
+    res = sorted(q.get(timeout=300) for _ in procs)
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    for run in range(2):
+        assert all(r[1][run][0] for r in res), "colouring differs from the oracle"
+        assert all(r[1][run][1] for r in res), "round count differs"
+        assert res[0][1][run][2] == res[1][1][run][2], "the ranks saw different round totals"
