@@ -75,6 +75,12 @@ constexpr bool kCountStream = GC_COUNT_STREAM != 0;
                        // instead of one thread per fresh vertex after the block's units
 #endif
 
+#ifndef GC_MERGED_HANDOFF
+#define GC_MERGED_HANDOFF 1  // 1: a block's item reservation IS its barrier arrival (one release
+                             // atomic), the staged items are copied while the barrier completes and
+                             // carry round tags the consumers check; 0: reserve, copy, then arrive
+#endif
+
 #ifndef GC_PACKED
 #define GC_PACKED 0  // 1: 32-bit (hi << 16 | lo) round counts -- max-min only (no JP / multi-hash branch);
                      // measured 27.9 vs 28.1 ms on R-MAT s24, not worth the restriction
@@ -106,7 +112,7 @@ constexpr uint32_t kInlineSeg = 4;         // schedule_fresh: rows of <= 4 segme
 constexpr int kHubChunk = 4096;
 constexpr uint32_t kFirst = 0x80000000u;   // item flag: colour v in this round
 constexpr uint32_t kLoSide = 0x40000000u;  // item flag: scheduled by its lo side (min colour)
-constexpr uint32_t kLenMask = 0x3FFFFFFFu;
+constexpr uint32_t kLenMask = GC_MERGED_HANDOFF ? 0x3FFu : 0x3FFFFFFFu;  // merged: bits 10-29 hold the round tag
 constexpr unsigned long long kDecHi = 0ull - (1ull << 32);
 // Packed counts: the rounds decrement a 32-bit word (hi << 16 | lo) per vertex
 // -- half the footprint of 64-bit words, so the round's burst of random
@@ -181,14 +187,23 @@ struct CArgs {
     int H;                         // MH: weight functions (count words v * H + j)
     uint32_t mkeys[GC_MAX_HASHES]; // MH: their keys K_j
     const uint32_t *dg;            // LDF: vertex degrees; nullptr = weights only
+    uint32_t epoch;                // colourings run on this handle (item round tags)
 };
+
+// Round tags of the items walked in round r (merged hand-off): items are
+// written after their producer's barrier arrival, so a consumer checks that
+// both 8-byte halves of an item carry round r's tag (each half is written by
+// one 8-byte element store, single-copy atomic) and re-reads until they do.
+// The epoch separates colourings (the arrays are cleared every 256).
+__device__ __forceinline__ uint32_t tag_a(uint32_t epoch, uint32_t r) { return ((epoch & 0xFu) << 16) | (r & 0xFFFFu); }
+__device__ __forceinline__ uint32_t tag_b(uint32_t epoch, uint32_t r) { return ((epoch & 0xFFu) << 16) | (r & 0xFFFFu); }
 
 // Priority key of v (R1; with LDF the (degree, weight) pair of R21 as one
 // 64-bit integer, degree in the high half): comparisons of keys are the
 // comparisons of Alg.5 L29-34 / Alg.2 L9.
 __device__ __forceinline__ uint64_t prio_key(const CArgs &a, uint32_t v) {
     const uint64_t w = weight_mix(v ^ a.key);
-    return a.dg ? w | ((uint64_t)__ldg(a.dg + v) << 32) : w;
+    return (a.dg && v != 0xFFFFFFFFu) ? w | ((uint64_t)__ldg(a.dg + v) << 32) : w;  // (kNone: a hole item)
 }
 // JP mex slot of a long row: a 1024-bit presence set of its predecessors'
 // colours + the number of its entries not yet walked (the segment that takes
@@ -297,7 +312,9 @@ __device__ __forceinline__ bool grid_barrier_rw(const CArgs &a, uint32_t k, int 
     __syncthreads();
     if (threadIdx.x == 0) {
         int ok = 1;
-#if GC_BARRIER_RELAXED_SPIN
+#if GC_MERGED_HANDOFF
+        // (the block arrived with its item reservation in stage_flush)
+#elif GC_BARRIER_RELAXED_SPIN
         // arrival without a return value (release pattern), relaxed spin,
         // one acquire fence after the last arrival is seen
         asm volatile("red.release.gpu.global.add.u64 [%0], %1;" ::"l"(round_word(a, slot, (int)(blockIdx.x % kNG))),
@@ -386,6 +403,7 @@ struct Stage {
     unsigned long long *rw;         // the next round's word R (item reservations, arrivals)
     unsigned long long nbase[2];    // where the next round's items start
     unsigned long long *ccol;       // coloured-count slot of this round
+    uint32_t tg_a, tg_b;            // round tags of the items appended now (next round's)
     unsigned long long rd[kNG];     // the groups' round words from the barrier
     unsigned long long gn[2][kNG + 1];  // per list: prefix of the groups' item counts of the round
     unsigned long long g0[2][kNG];  // per list and group: where the round's items start
@@ -429,6 +447,44 @@ __device__ __forceinline__ const Item *round_item(const CArgs &a, int li, unsign
            (t - st.gn[li][gq]);
 }
 
+// an item of the next round into global memory (tagged under the merged hand-off)
+__device__ __forceinline__ void gput(Item *p, const Item &v) {
+#if GC_MERGED_HANDOFF
+    const Stage &st = stage();
+    // (a hole's lf / e0 may be uninitialised shared memory: masked to their fields)
+    const unsigned long long w0 =
+        (unsigned long long)v.v | ((unsigned long long)((v.lf & 0xC00003FFu) | (st.tg_a << 10)) << 32);
+    const unsigned long long w1 = ((unsigned long long)v.e0 & ((1ull << 40) - 1ull)) | ((unsigned long long)st.tg_b << 40);
+    asm volatile("st.relaxed.gpu.global.v2.u64 [%0], {%1, %2};" ::"l"(p), "l"(w0), "l"(w1) : "memory");
+#else
+    *p = v;
+#endif
+}
+// an item of round k (merged hand-off: until both halves carry its tags)
+__device__ __forceinline__ Item gget(const CArgs &a, const Item *p, uint32_t k) {
+    Item it;
+#if GC_MERGED_HANDOFF
+    const uint32_t ta = tag_a(a.epoch, k), tb = tag_b(a.epoch, k);
+    unsigned long long w0, w1;
+    for (unsigned spins = 0;; ++spins) {
+        asm volatile("ld.relaxed.gpu.global.v2.u64 {%0, %1}, [%2];" : "=l"(w0), "=l"(w1) : "l"(p) : "memory");
+        if ((((uint32_t)(w0 >> 32) >> 10) & 0xFFFFFu) == ta && (uint32_t)(w1 >> 40) == tb) break;
+        if (spins > (1u << 24)) {  // ~seconds: an item that never arrives (cannot happen)
+            flag_error(a, 11, k, (uint32_t)w0);
+            break;
+        }
+    }
+    it.v = (uint32_t)w0;
+    it.lf = (uint32_t)(w0 >> 32) & ~(0xFFFFFu << 10);
+    it.e0 = (int64_t)(w1 & ((1ull << 40) - 1ull));
+#else
+    (void)a;
+    (void)k;
+    it = *p;
+#endif
+    return it;
+}
+
 // Whole warp converged: lanes with `pred` append `val` to staged list li;
 // beyond the shared capacity the entries go straight to the global list.
 __device__ __forceinline__ void stage_append(const CArgs &a, bool pred, const Item &val, int li) {
@@ -454,7 +510,7 @@ __device__ __forceinline__ void stage_append(const CArgs &a, bool pred, const It
         if (spill) {
             const unsigned long long at = st.nbase[li] + gb + __popc(sm & ((1u << lane) - 1u));
             const unsigned long long capg = li == 0 ? a.sl_cap : a.wl_cap;
-            if (at < capg) (li == 0 ? a.SL + grp_base(a, 0) : a.WL + grp_base(a, 1))[at] = val;
+            if (at < capg) gput((li == 0 ? a.SL + grp_base(a, 0) : a.WL + grp_base(a, 1)) + at, val);
             else flag_error(a, 1, 0, val.v);
         }
     }
@@ -479,8 +535,17 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
     if (threadIdx.x == 0) {
         // both reservations in flight together (each is an L2 round trip)
         const unsigned c0 = min(st.n[0], (unsigned)kStS), c1 = min(st.n[1], (unsigned)kStW);
+        if (st.colored) atom_add_global(st.ccol, (unsigned long long)st.colored);  // before the arrival
+        st.colored = 0;
+#if GC_MERGED_HANDOFF
+        // one reservation for both lists, which is also the barrier arrival:
+        // the release orders every earlier write of the block (colours, Z
+        // stamps, spilled items); the staged items follow, tagged
+        const unsigned long long rv = atom_add_release(st.rw, rw_add(c0, 0) + rw_add(c1, 1) + kRwArr);
+#else
         // one reservation for both lists
         const unsigned long long rv = (c0 || c1) ? atom_add_global(st.rw, rw_add(c0, 0) + rw_add(c1, 1)) : 0ull;
+#endif
         if (GC_PROF_FRESH && prs) {  // the reservation came back
             asm volatile("" ::"l"(rv));
             red_max(prs + 9, gtimer() - t_round);
@@ -499,13 +564,11 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
             }
         }
         st.nf = 0;
-        if (st.colored) atom_add_global(st.ccol, (unsigned long long)st.colored);
-        st.colored = 0;
     }
     __syncthreads();
     Item *const sl = a.SL + grp_base(a, 0), *const wl = a.WL + grp_base(a, 1);
-    for (unsigned i = threadIdx.x; i < st.n[0]; i += blockDim.x) sl[st.base[0] + i] = st.s[i];
-    for (unsigned i = threadIdx.x; i < st.n[1]; i += blockDim.x) wl[st.base[1] + i] = st.w[i];
+    for (unsigned i = threadIdx.x; i < st.n[0]; i += blockDim.x) gput(sl + st.base[0] + i, st.s[i]);
+    for (unsigned i = threadIdx.x; i < st.n[1]; i += blockDim.x) gput(wl + st.base[1] + i, st.w[i]);
     __syncthreads();
     if (threadIdx.x < 2) st.n[threadIdx.x] = 0;
     if (prs && threadIdx.x == 0)
@@ -943,7 +1006,7 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
                 st.s[pos] = it;
             } else {
                 const unsigned long long at = st.nbase[0] + rw_field(atom_add_global(st.rw, 1ull), 0);
-                if (at < a.sl_cap) a.SL[grp_base(a, 0) + at] = it;
+                if (at < a.sl_cap) gput(a.SL + grp_base(a, 0) + at, it);
                 else flag_error(a, 1, 0, f.x);
             }
         } else {
@@ -974,7 +1037,7 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
                     si.e0 = rs + (int64_t)q * kSeg;
                     si.lf = (uint32_t)min((int64_t)kSeg, len - (int64_t)q * kSeg) | ((q == 0 || (JP && a.jpv == 1)) ? fl : 0u);
                     if (dst >= 0) st.w[dst + q] = si;
-                    else a.WL[grp_base(a, 1) + ~dst + q] = si;
+                    else gput(a.WL + grp_base(a, 1) + ~dst + q, si);
                 }
             }
         }
@@ -991,7 +1054,7 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
             si.e0 = L.rs + (int64_t)q * kSeg;
             si.lf = (uint32_t)min((int64_t)kSeg, (int64_t)L.len - (int64_t)q * kSeg) | ((q == 0 || (JP && a.jpv == 1)) ? L.flags : 0u);
             if (L.dst >= 0) st.w[L.dst + q] = si;
-            else a.WL[grp_base(a, 1) + ~L.dst + q] = si;
+            else gput(a.WL + grp_base(a, 1) + ~L.dst + q, si);
             if (GC_PREFETCH_WL) {  // the segment walked next round: HBM -> L2 now
                 const uint32_t ln = si.lf & kLenMask;
                 for (uint32_t o = 0; o < ln; o += 32) asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ci + si.e0 + o));
@@ -1143,6 +1206,8 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
         // count for round 0 (so the "next round" targets are round 0's here)
         if (threadIdx.x == 0) {
             st.rw = round_word(a, 0, (int)(blockIdx.x % kNG));  // round 0's word
+            st.tg_a = tag_a(a.epoch, 0u);
+            st.tg_b = tag_b(a.epoch, 0u);
             st.nbase[0] = st.nbase[1] = 0ull;
             st.ccol = a.ctr + cK;
         }
@@ -1247,6 +1312,8 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
             }
             st.trap = (k & 31u) == 0u ? __ldcg(&a.ctr[cErr]) : 0ull;
             st.rw = round_word(a, (int)((k + 1) % 3), me);
+            st.tg_a = tag_a(a.epoch, k + 1u);
+            st.tg_b = tag_b(a.epoch, k + 1u);
             st.ccol = a.ctr + cK + 16 * cur;
         }
         __syncthreads();
@@ -1276,7 +1343,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
             const long long c_unit = PROF ? clock64() : 0;
             if (u < nw) {
                 // longer rows: one <= kSeg-entry item per warp
-                Item it = *round_item(a, 1, u);
+                Item it = gget(a, round_item(a, 1, u), k);
                 if (it.v == kNone) it.lf = 0;  // hole left by schedule_fresh
                 const uint64_t pv = prio_key(a, it.v);
                 if (JP && a.jpv != 1) {  // Alg.2 / Alg.4: the colour is the round (remapped for Alg.4)
@@ -1330,7 +1397,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                 bool want = false, cl = false;
                 uint32_t lf = 0, z = 0;
                 if (idx < ns) {
-                    const Item it = *round_item(a, 0, idx);
+                    const Item it = gget(a, round_item(a, 0, idx), k);
                     v = it.v;
                     lf = it.lf;
                     len = it.lf & kLenMask;
@@ -1364,7 +1431,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                 bool want = false, cl = false;
                 uint32_t lf = 0, z = 0;
                 if (idx < ns) {
-                    const Item it = *round_item(a, 0, idx);
+                    const Item it = gget(a, round_item(a, 0, idx), k);
                     v = it.v;
                     lf = it.lf;
                     len = it.lf & kLenMask;
@@ -1825,6 +1892,10 @@ int ensure_count_scratch(gc_graph *g) {
     // one monotone array per barrier group (each could receive every item)
     GC_CUDA_TRY(dmalloc(&s.SL, (size_t)kNG * (size_t)s.sl_cap * sizeof(Item)));
     GC_CUDA_TRY(dmalloc(&s.WL, (size_t)kNG * (size_t)s.wl_cap * sizeof(Item)));
+    // (recycled memory could hold tagged items of another handle's colouring)
+    GC_CUDA_TRY(cudaMemsetAsync(s.SL, 0, (size_t)kNG * (size_t)s.sl_cap * sizeof(Item), g->stream));
+    GC_CUDA_TRY(cudaMemsetAsync(s.WL, 0, (size_t)kNG * (size_t)s.wl_cap * sizeof(Item), g->stream));
+    s.count_epoch = 0;
     // hub chunk list: at most nnz / kHubChunk entries
     GC_CUDA_TRY(dmalloc(&s.hubs, ((size_t)g->nnz / kHubChunk + 1) * 8));
     GC_CUDA_TRY(dmalloc(&s.cctr, kCCtrWords * sizeof(unsigned long long)));
@@ -1972,6 +2043,15 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
     a.H = p.H;
     for (int j = 0; j < GC_MAX_HASHES; ++j) a.mkeys[j] = p.keys.k[j];
     a.dg = dg;
+    // item round tags (merged hand-off): a new epoch per colouring; the item
+    // arrays are cleared when the 8-bit epoch wraps (a stale item then
+    // cannot carry a current tag); epoch 0 (the cleared state) is never used
+    if (++s.count_epoch % 256u == 0u) {
+        GC_CUDA_TRY(cudaMemsetAsync(s.SL, 0, (size_t)kNG * (size_t)s.sl_cap * sizeof(Item), st));
+        GC_CUDA_TRY(cudaMemsetAsync(s.WL, 0, (size_t)kNG * (size_t)s.wl_cap * sizeof(Item), st));
+        ++s.count_epoch;
+    }
+    a.epoch = s.count_epoch;
     a.M = s.cM;
     a.jpv = jpv;
     a.cr = nullptr;

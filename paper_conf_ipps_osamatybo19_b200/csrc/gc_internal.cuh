@@ -74,6 +74,7 @@ struct Scratch {
     uint32_t *hubs = nullptr;            // k_count: rows counted by blocks
     unsigned long long *cctr = nullptr;  // counters of the persistent count kernel
     int64_t sl_cap = 0, wl_cap = 0;
+    uint32_t count_epoch = 0;            // COUNT colourings run (item round tags, gc_count.cu)
     uint32_t *cM = nullptr;              // COUNT mode: status bits (1 = uncoloured)
     uint32_t *crow = nullptr;            // COUNT mode: row of each counting chunk's first entry
     int64_t nch = 0;
