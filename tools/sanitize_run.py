@@ -27,6 +27,8 @@ CASES = [
     ("is_alg2", gcb.IS_ALG2, gcb.MODE_COUNT, lambda g: O.color_is_alg2(g, 1)),
     ("jp_alg4", gcb.JP_ALG4, gcb.MODE_COUNT, lambda g: O.color_jp_alg4(g, 1)),
     ("hash_is8", gcb.HASH_IS(8), gcb.MODE_AUTO, lambda g: O.color_hash_is(g, 1, 8)),
+    ("maxmin_ldf", gcb.LDF(gcb.MAXMIN), gcb.MODE_COUNT, lambda g: O.color_maxmin(g, 1, ldf=True)),
+    ("luby_ldf", gcb.LDF(gcb.LUBY_MIS), gcb.MODE_COUNT, lambda g: O.color_luby(g, 1, ldf=True)),
 ]
 
 
@@ -40,6 +42,15 @@ def main():
                 _, k, st = h.color(1, v, out, mode=mode, stats=True)
                 ok = (out.cpu().numpy().view(np.uint32) == ref(g)).all()
                 print(f"{cfg} {name} mode {st.mode_used}: colours {k} rounds {st.rounds} "
+                      f"{'ok' if ok else 'MISMATCH'}", flush=True)
+                assert ok
+        # the partitioned kernel (device-driven rounds), 2 and 3 partitions on this GPU
+        for parts in (2, 3):
+            with gcb.loopback_graph(g.n, g.row_offsets, g.col_indices, parts) as h:
+                out = torch.empty(g.n, dtype=torch.int32, device="cuda")
+                _, k, st = h.color(1, gcb.MAXMIN, out, stats=True)
+                ok = (out.cpu().numpy().view(np.uint32) == O.color_maxmin(g, 1)).all()
+                print(f"{cfg} maxmin loopback P={parts}: colours {k} rounds {st.rounds} "
                       f"{'ok' if ok else 'MISMATCH'}", flush=True)
                 assert ok
 
