@@ -42,7 +42,7 @@ constexpr int64_t kChunk = 1024;
 constexpr unsigned long long kDecHi = 0ull - (1ull << 32);
 constexpr unsigned long long kDecLo = ~0ull;
 
-enum : int { cSEnd = 0, cLo, cHi, cPairs, cLong, cErr, cErrV, cChunks, cTicket, kDCtrWords = 16 };
+enum : int { cSEnd = 0, cLo, cHi, cPairs, cLong, cErr, cErrV, cChunks, cTicket, kDCtrWords = 24 };
 
 struct LongJob {
     int64_t s, e;     // entry range
@@ -415,22 +415,27 @@ __device__ __forceinline__ bool group_barrier(unsigned long long *ctr, unsigned 
     return ok_sh != 0;
 }
 
-__device__ __forceinline__ void dec_k(const DCArgs &a, uint32_t pv, uint32_t lw, uint32_t wg, uint32_t k) {
-    const bool hi = pv > weight_mix(wg ^ a.key);
-    const unsigned long long old = atomicAdd(a.cnt + lw, hi ? kDecHi : kDecLo);
-    const uint32_t side = hi ? (uint32_t)(old >> 32) : (uint32_t)old;
-    const uint32_t other = hi ? (uint32_t)old : (uint32_t)(old >> 32);
-    if (side == 1u) {
-        if (other != 0u) push_s(a, lw | (hi ? 0u : kLoF));
-        else if (!hi) a.Z[lw] = k + 1u;
-    } else if (side == 0u) {
-        flag(a, 4, wg);
-    }
-}
 // entries [s, e) of an own row (global ids; remote ones skipped) or a ghost
 // row (owned ids), lanes `sub` of `width`; kQ entries per lane in flight (the
 // atomics of a batch are issued together, not one round trip per entry)
 constexpr int kQ = 4;
+// device-driven rounds keep two scheduled lists, S[0, n_loc) and
+// S[n_loc, 2 n_loc): a vertex freed in round k goes to list (k+1) % 2, whose
+// length (ctr[cSL + (k+1) % 2]) is final at the round-end barrier and is not
+// touched by round k+1's pushes -- every block reads the same round slice
+// even when a fast block is already freeing round-(k+2) vertices
+enum : int { cSL = 16 };  // [list] lengths (DCState ctr)
+__device__ __forceinline__ void push_sk(const DCArgs &a, uint32_t val, uint32_t k) {
+    const unsigned lst = (k + 1u) & 1u;
+    const unsigned m = __activemask();
+    const int leader = __ffs(m) - 1;
+    unsigned long long base = 0;
+    if ((int)lane_id() == leader) base = atomicAdd(a.ctr + cSL + lst, (unsigned long long)__popc(m));
+    base = __shfl_sync(m, base, leader);
+    const unsigned long long at = base + __popc(m & ((1u << lane_id()) - 1u));
+    if (at < (unsigned long long)a.n_loc) a.S[(int64_t)lst * a.n_loc + (int64_t)at] = val;
+    else flag(a, 2, val);
+}
 template <bool GHOST>
 __device__ __forceinline__ void walk_entries_k(const DCArgs &a, uint32_t pv, int64_t s, int64_t e, int64_t sub,
                                                int64_t width, uint32_t k) {
@@ -463,7 +468,7 @@ __device__ __forceinline__ void walk_entries_k(const DCArgs &a, uint32_t pv, int
             const uint32_t side = hi[q] ? (uint32_t)(old[q] >> 32) : (uint32_t)old[q];
             const uint32_t other = hi[q] ? (uint32_t)old[q] : (uint32_t)(old[q] >> 32);
             if (side == 1u) {
-                if (other != 0u) push_s(a, lw[q] | (hi[q] ? 0u : kLoF));
+                if (other != 0u) push_sk(a, lw[q] | (hi[q] ? 0u : kLoF), k);
                 else if (!hi[q]) a.Z[lw[q]] = k + 1u;
             } else if (side == 0u) {
                 flag(a, 4, wg[q]);
@@ -524,6 +529,7 @@ __global__ void __launch_bounds__(256) k_dc_persistent(const __grid_constant__ D
     __shared__ unsigned long long peer_cnt[kMaxWorld];
     __shared__ unsigned long long sh_tot, sh_err, sh_nrecv;
     int64_t remaining = A.n_global;
+    // round 0: the counting pass's list S[cLo, cHi); round k >= 1: list k % 2
     int64_t lo = (int64_t)__ldcg(a.ctr + cLo), hi = (int64_t)__ldcg(a.ctr + cHi);
     uint32_t k = 0;
     unsigned long long err_out = 0;
@@ -539,7 +545,7 @@ __global__ void __launch_bounds__(256) k_dc_persistent(const __grid_constant__ D
         }
         // A. own scheduled vertices
         for (int64_t i = lo + gid; i < hi; i += ng) {
-            const uint32_t it = a.S[i];
+            const uint32_t it = a.S[(k ? (int64_t)par * a.n_loc : 0) + i];
             const uint32_t lv = it & ~kLoF;
             const uint32_t vg = a.v0 + lv;
             const int64_t rs = a.ro[lv], re = a.ro[lv + 1];
@@ -566,6 +572,9 @@ __global__ void __launch_bounds__(256) k_dc_persistent(const __grid_constant__ D
         // other partitions' mailbox words are in flight (E1)
         const unsigned long long n_own = __ldcg(a.ctr + cChunks2 + par);
         const unsigned long long own = __ldcg(a.ctr + cPairs2 + par);
+        // list par was consumed in A (all blocks passed barrier 1): reset its
+        // length for round k+1's pushes (ordered before them by barrier 3)
+        if (k && gb == 0 && threadIdx.x == 0) a.ctr[cSL + par] = 0ull;
         if (gb == 0 && threadIdx.x == 0 && A.world > 1) {
             const unsigned long long e = __ldcg(a.ctr + cErr) ? 1ull : 0ull;
             const unsigned long long w = mbox_word(A.epoch, k, own, e);
@@ -656,16 +665,18 @@ __global__ void __launch_bounds__(256) k_dc_persistent(const __grid_constant__ D
             }
         }
         if (tl) atomicMax(tl + 3, gtimer_dp() - t_round);  // ghost walks done
-        if (!group_barrier(bar, gsize, ++nbar)) { err_out = 5; break; }
-        if (tl) atomicMax(tl + 4, gtimer_dp() - t_round);  // group barrier 2
-        // E2. the chunks of long ghost rows (queued after the own ones)
-        walk_chunks(a, true, 0, __ldcg(a.ctr + cGChunks2 + par), gb, gsize, k);
+        if (A.world > 1) {  // (one partition: no ghost rows, nothing queued here)
+            if (!group_barrier(bar, gsize, ++nbar)) { err_out = 5; break; }
+            if (tl) atomicMax(tl + 4, gtimer_dp() - t_round);  // group barrier 2
+            // E2. the chunks of long ghost rows (queued after the own ones)
+            walk_chunks(a, true, 0, __ldcg(a.ctr + cGChunks2 + par), gb, gsize, k);
+        }
         if (tl) atomicMax(tl + 5, gtimer_dp() - t_round);  // long chunks done
         if (!group_barrier(bar, gsize, ++nbar)) { err_out = 5; break; }
         if (tl) atomicMax(tl + 6, gtimer_dp() - t_round);  // group barrier 3 (round end)
         remaining -= (int64_t)tot;
-        lo = hi;
-        hi = (int64_t)__ldcg(a.ctr + cSEnd);
+        lo = 0;
+        hi = (int64_t)__ldcg(a.ctr + cSL + npar);
         if (remaining <= 0) {
             ++k;
             break;
@@ -740,7 +751,7 @@ int ensure_dc(gc_graph *g, Part &p, int64_t n_global) {
     if (!s.cnt) {
         GC_CUDA_TRY(dmalloc(&s.cnt, nl * 8));
         GC_CUDA_TRY(dmalloc(&s.Z, nl * 4));
-        GC_CUDA_TRY(dmalloc(&s.S, nl * 4));
+        GC_CUDA_TRY(dmalloc(&s.S, 2 * nl * 4));  // two lists (device-driven rounds)
         // long jobs of one round: own rows and ghost rows longer than kLongMin
         // (each at most nnz / kLongMin); chunk items: at most 2 nnz / kChunk + jobs
         s.L_cap = 2 * (p.nnz / std::min(kLongMin, kPLongMin)) + 16;  // own + ghost rows longer than the threshold

@@ -497,6 +497,21 @@ def test_loopback_count_hubs_and_ghost_rows(parts):
             assert st.rounds == R and st.frontier_sizes == nk
 
 
+@pytest.mark.parametrize("parts", [3, 4, 8])
+def test_loopback_repeated_colourings_stable(parts):
+    """Device-driven partitioned rounds repeated back to back (a race between
+    a fast block freeing round-(k+2) vertices and a slow block reading round
+    k+1's scheduled slice once showed up only after several colourings): 24
+    colourings of one handle, each equal to the oracle."""
+    g = G.rmat(18, 16, seed=11)
+    ref = O.color_maxmin(g, 2)
+    with gcb.loopback_graph(g.n, g.row_offsets, g.col_indices, parts) as h:
+        out = torch.empty(g.n, dtype=torch.int32)
+        for i in range(24):
+            h.color(2, gcb.MAXMIN, out, mode=gcb.MODE_COUNT)
+            assert (out.numpy().view(np.uint32) == ref).all(), (parts, i)
+
+
 def test_cfg5_style_partitioned_rmat_s25():
     """cfg5's check at the largest size a test affords: R-MAT s25 (1.08e9
     entries) partitioned P = 2, 4 (loopback transport: the same COUNT rounds,
