@@ -81,6 +81,12 @@ constexpr bool kCountStream = GC_COUNT_STREAM != 0;
                              // carry round tags the consumers check; 0: reserve, copy, then arrive
 #endif
 
+#ifndef GC_SKIP_DEAD
+#define GC_SKIP_DEAD 1  // 1: max-min walks skip the neighbours on the vertex's scheduling side
+                        // (all coloured before its round: their counts are dead), see walk()
+#endif
+constexpr bool kSkipDead = GC_SKIP_DEAD != 0;
+
 #ifndef GC_PACKED
 #define GC_PACKED 0  // 1: 32-bit (hi << 16 | lo) round counts -- max-min only (no JP / multi-hash branch);
                      // measured 27.9 vs 28.1 ms on R-MAT s24, not worth the restriction
@@ -623,7 +629,7 @@ __device__ __forceinline__ void schedule_rows(const CArgs &a, bool pred, uint32_
             si.v = ww;
             const int64_t e0 = r0 + (int64_t)q * kSeg;
             si.e0 = e0;
-            si.lf = (uint32_t)min((int64_t)kSeg, r0 + ln - e0) | ((q == 0 || (JP && a.jpv == 1)) ? fs : 0u);
+            si.lf = (uint32_t)min((int64_t)kSeg, r0 + ln - e0) | ((q == 0 || (JP && a.jpv == 1)) ? fs : (fs & kLoSide));
             stage_append(a, q < nseg, si, 1);
         }
     }
@@ -658,7 +664,7 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint64_t pv, in
                                      int64_t end, int stride, uint32_t k, uint32_t &nvis,
                                      unsigned long long *mask = nullptr, uint32_t *sbits = nullptr,
                                      bool want_mex = false, bool want_set = false,
-                                     long long *tprof = nullptr) {
+                                     long long *tprof = nullptr, int skipside = -1) {
     uint32_t w[Q];
 #pragma unroll
     for (int q = 0; q < Q; ++q) {
@@ -690,11 +696,21 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint64_t pv, in
     uint32_t cv[Q];  // JP: colours of the larger neighbours
 #pragma unroll
     for (int q = 0; q < Q; ++q) {
-        const bool live = w[q] != kNone;
+        bool live = w[q] != kNone;
         const uint32_t wq = live ? w[q] : 0u;
         // v is a larger neighbour of w (LDF: the degree decides first, R21)
         hi[q] = live && pv > ((uint64_t)weight_mix(wq ^ a.key) | (a.dg ? (uint64_t)__ldg(a.dg + wq) << 32 : 0ull));
         cv[q] = kNone;
+        // dead side (max-min): v's scheduling side was free at the start of
+        // this round, so every neighbour on that side was coloured in an
+        // earlier round and its counts decide nothing any more -- no atomic
+        // (skipside 0: v freed by its hi side, its larger neighbours are dead;
+        // 1: by its lo side, its smaller ones).  Decrements to uncoloured
+        // vertices are never skipped, so the schedule is unchanged.
+        if (kSkipDead && !JP && live && skipside >= 0 && hi[q] == (skipside == 1)) {
+            w[q] = kNone;
+            live = false;
+        }
 #if GC_PACKED
         slot[q] = (live && a.nbig > 0) ? big_slot(wq) : -1;
         uint32_t *adr = slot[q] >= 0 ? a.big32 + 2 * slot[q] + (hi[q] ? 0 : 1) : a.cnt32 + wq;
@@ -1035,7 +1051,7 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
                     Item si;
                     si.v = f.x;
                     si.e0 = rs + (int64_t)q * kSeg;
-                    si.lf = (uint32_t)min((int64_t)kSeg, len - (int64_t)q * kSeg) | ((q == 0 || (JP && a.jpv == 1)) ? fl : 0u);
+                    si.lf = (uint32_t)min((int64_t)kSeg, len - (int64_t)q * kSeg) | ((q == 0 || (JP && a.jpv == 1)) ? fl : (fl & kLoSide));
                     if (dst >= 0) st.w[dst + q] = si;
                     else gput(a.WL + grp_base(a, 1) + ~dst + q, si);
                 }
@@ -1052,7 +1068,7 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
             Item si;
             si.v = L.w;
             si.e0 = L.rs + (int64_t)q * kSeg;
-            si.lf = (uint32_t)min((int64_t)kSeg, (int64_t)L.len - (int64_t)q * kSeg) | ((q == 0 || (JP && a.jpv == 1)) ? L.flags : 0u);
+            si.lf = (uint32_t)min((int64_t)kSeg, (int64_t)L.len - (int64_t)q * kSeg) | ((q == 0 || (JP && a.jpv == 1)) ? L.flags : (L.flags & kLoSide));
             if (L.dst >= 0) st.w[L.dst + q] = si;
             else gput(a.WL + grp_base(a, 1) + ~L.dst + q, si);
             if (GC_PREFETCH_WL) {  // the segment walked next round: HBM -> L2 now
@@ -1265,7 +1281,8 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
             if (lane == 0) a.M[base >> 5] = live;
         }
         if (lane == 0 && word) atomicAdd(&stage().colored, (unsigned)__popc(word));
-        schedule_rows<JP>(a, zero && re > rs, v, rs, re - rs, 0u);  // walked in round 0
+        // walked in round 0 (the free side's flag: its neighbours, if any, are dead)
+        schedule_rows<JP>(a, zero && re > rs, v, rs, re - rs, (!JP && !MH && lo == 0u) ? kLoSide : 0u);
     }
     stage_flush(a);
     if (!grid_barrier_rw(a, 0, 0, stage().rd)) return;
@@ -1372,7 +1389,8 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                         walk_mh<kSeg / 32>(a, it.v, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k, nvis);
                     else
                         walk<kSeg / 32, JP>(a, it.v, pv, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k, nvis,
-                                            nullptr, nullptr, false, false, (GC_PROF_UNIT && prs) ? tp : nullptr);
+                                            nullptr, nullptr, false, false, (GC_PROF_UNIT && prs) ? tp : nullptr,
+                                            JP ? -1 : ((it.lf & kLoSide) ? 1 : 0));
                     if (cl) colour_fin<MH>(a, it.v, it.lf, k, z);
                     if (GC_PROF_UNIT && prs && !MH) {
                         // max over the warp's lanes of each stage's end (cycles since the unit start)
@@ -1415,7 +1433,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                 for (uint32_t j = 0; __any_sync(kFull, j < len); j += 4) {
                     if (MH) walk_mh<4>(a, j < len ? v : kNone, e0 + j, e0 + len, 1, k, nvis);
                     else walk<4, JP>(a, j < len ? v : kNone, pv, e0 + j, e0 + len, 1, k, nvis, &mask, nullptr, want,
-                                     JP && a.jpv == 3);
+                                     JP && a.jpv == 3, nullptr, JP ? -1 : ((lf & kLoSide) ? 1 : 0));
                 }
                 if (cl) colour_fin<MH>(a, v, lf, k, z);
                 if (JP && want) {  // <= 32 predecessors: the mex is below 64
@@ -1448,7 +1466,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                 unsigned long long mask = 0ull;
                 if (MH) walk_mh<4>(a, v, e0 + (lane & 7u), e0 + len, 8, k, nvis);
                 else walk<4, JP>(a, v, pv, e0 + (lane & 7u), e0 + len, 8, k, nvis, &mask, nullptr, want,
-                                 JP && a.jpv == 3);
+                                 JP && a.jpv == 3, nullptr, JP ? -1 : ((lf & kLoSide) ? 1 : 0));
                 if (cl) colour_fin<MH>(a, v, lf, k, z);
                 if (JP && a.jpv == 1) {
                     mask = group8_or(mask);
