@@ -87,6 +87,13 @@ constexpr bool kCountStream = GC_COUNT_STREAM != 0;
 #endif
 constexpr bool kSkipDead = GC_SKIP_DEAD != 0;
 
+#ifndef GC_RELAXED_ARRIVE
+#define GC_RELAXED_ARRIVE 1  // 1: max-min / multi-hash rounds k >= 1 arrive with a relaxed atomic and
+                             // leave the barrier without an acquire fence (see stage_flush)
+#endif
+constexpr bool kRelaxedArrive = GC_RELAXED_ARRIVE != 0;
+
+
 #ifndef GC_PACKED
 #define GC_PACKED 0  // 1: 32-bit (hi << 16 | lo) round counts -- max-min only (no JP / multi-hash branch);
                      // measured 27.9 vs 28.1 ms on R-MAT s24, not worth the restriction
@@ -150,6 +157,7 @@ enum : int {
     cK = 96,        // [96, 112, 128]: vertices coloured in the round (stats)
     cCol = 144,     // vertices coloured (written at the end, host check)
     cBar = 160,     // (unused: arrivals live in the round words)
+    cFin = 168,     // relaxed rounds: the final release / acquire barrier
     cAbort = 176,
     cErr = 192,     // [192..194] first trap: kind, round, vertex
     cRounds = 208,  // result: rounds R
@@ -313,7 +321,7 @@ __device__ __forceinline__ unsigned group_size(int grp) {
     return (gridDim.x - (unsigned)grp + kNG - 1) / kNG;
 }
 __device__ __forceinline__ bool grid_barrier_rw(const CArgs &a, uint32_t k, int slot,
-                                                unsigned long long *out) {
+                                                unsigned long long *out, bool acquire = true) {
     __shared__ int ok_sh;
     __syncthreads();
     if (threadIdx.x == 0) {
@@ -343,7 +351,7 @@ __device__ __forceinline__ bool grid_barrier_rw(const CArgs &a, uint32_t k, int 
             }
             if (done) {
 #if GC_BARRIER_RELAXED_SPIN
-                asm volatile("fence.acq_rel.gpu;" ::: "memory");
+                if (acquire) asm volatile("fence.acq_rel.gpu;" ::: "memory");
 #endif
                 break;
             }
@@ -524,8 +532,13 @@ __device__ __forceinline__ void stage_append(const CArgs &a, bool pred, const It
 
 // Whole block: move staged items to the global lists, add the coloured count.
 // PROF: prs = this round's stat record (entries walked, longest block work).
+// relaxed (max-min rounds k >= 1): the arrival needs no release because no
+// later round reads anything the round writes through a plain load: items
+// carry round tags and are re-read until both halves do, the counts are
+// atomics, and the lo-freed-second stamps and the colours are read only after
+// the rounds, behind one release / acquire barrier (colour_final).
 __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullptr,
-                                            unsigned long long t_round = 0) {
+                                            unsigned long long t_round = 0, bool relaxed = false) {
     Stage &st = stage();
     __syncthreads();
     if (prs && threadIdx.x == 0) {
@@ -541,13 +554,16 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
     if (threadIdx.x == 0) {
         // both reservations in flight together (each is an L2 round trip)
         const unsigned c0 = min(st.n[0], (unsigned)kStS), c1 = min(st.n[1], (unsigned)kStW);
-        if (st.colored) atom_add_global(st.ccol, (unsigned long long)st.colored);  // before the arrival
+        // the round's coloured count (statistics: the frontier trace; under
+        // relaxed arrivals the completion check counts the colours instead)
+        if (st.colored) atom_add_global(st.ccol, (unsigned long long)st.colored);
         st.colored = 0;
 #if GC_MERGED_HANDOFF
         // one reservation for both lists, which is also the barrier arrival:
         // the release orders every earlier write of the block (colours, Z
         // stamps, spilled items); the staged items follow, tagged
-        const unsigned long long rv = atom_add_release(st.rw, rw_add(c0, 0) + rw_add(c1, 1) + kRwArr);
+        const unsigned long long rv = relaxed ? atom_add_global(st.rw, rw_add(c0, 0) + rw_add(c1, 1) + kRwArr)
+                                              : atom_add_release(st.rw, rw_add(c0, 0) + rw_add(c1, 1) + kRwArr);
 #else
         // one reservation for both lists
         const unsigned long long rv = (c0 || c1) ? atom_add_global(st.rw, rw_add(c0, 0) + rw_add(c1, 1)) : 0ull;
@@ -777,7 +793,7 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint64_t pv, in
             }
             if (side == 1u) {
                 if (other != 0u) fresh[q] = true;        // first side freed: schedule w
-                else if (!hi[q]) a.Zlo[w[q]] = k + 1u;   // lo freed second
+                else if (!hi[q]) a.Zlo[w[q]] = k + 1u;   // lo freed second (read after the rounds)
             } else if (side == 0u) {
                 flag_error(a, 4, k, w[q]);  // count underflow: adjacency not symmetric
             }
@@ -1194,6 +1210,10 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
     const unsigned long long nthreads = (unsigned long long)gridDim.x * blockDim.x;
     const unsigned long long gwarp = gtid >> 5, nwarps = nthreads >> 5;
     const int64_t n = a.n;
+    // max-min: rounds k >= 1 end with relaxed arrivals; the colours written
+    // in the rounds are provisional (max unless the item's side is lo) and
+    // the lo-freed-second stamps are applied after the rounds (colour_final)
+    constexpr bool kRelax = kRelaxedArrive && !JP && !MH;
     uint32_t nvis = 0;
     unsigned long long nvis_tot = 0, t_rounds = 0;
     unsigned long long t0 = PROF ? gtimer() : 0ull;
@@ -1379,7 +1399,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                     jp_segment_done(a, it.v, it.lf & kLenMask, pv, sb, k);
                 } else {
                     const bool cl = !JP && (it.lf & kFirst) && lane == 0;
-                    const uint32_t z = cl ? __ldcg(a.Zlo + it.v) : 0u;
+                    const uint32_t z = (cl && !kRelax) ? __ldcg(a.Zlo + it.v) : kNever;
                     long long tp[3] = {0, 0, 0};
                     if (GC_PROF_UNIT && prs) {
                         asm volatile("" ::"l"(pv));
@@ -1413,7 +1433,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                 uint64_t pv = 0;
                 int64_t e0 = 0;
                 bool want = false, cl = false;
-                uint32_t lf = 0, z = 0;
+                uint32_t lf = 0, z = kNever;
                 if (idx < ns) {
                     const Item it = gget(a, round_item(a, 0, idx), k);
                     v = it.v;
@@ -1427,7 +1447,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                         atomicAdd(&stage().colored, 1u);
                     }
                     cl = !JP && (it.lf & kFirst);
-                    if (cl) z = __ldcg(a.Zlo + v);
+                    if (cl && !kRelax) z = __ldcg(a.Zlo + v);
                 }
                 unsigned long long mask = 0ull;
                 for (uint32_t j = 0; __any_sync(kFull, j < len); j += 4) {
@@ -1447,7 +1467,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                 uint64_t pv = 0;
                 int64_t e0 = 0;
                 bool want = false, cl = false;
-                uint32_t lf = 0, z = 0;
+                uint32_t lf = 0, z = kNever;
                 if (idx < ns) {
                     const Item it = gget(a, round_item(a, 0, idx), k);
                     v = it.v;
@@ -1461,7 +1481,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
                         atomicAdd(&stage().colored, 1u);
                     }
                     cl = !JP && (it.lf & kFirst) && (lane & 7u) == 0u;
-                    if (cl) z = __ldcg(a.Zlo + v);
+                    if (cl && !kRelax) z = __ldcg(a.Zlo + v);
                 }
                 unsigned long long mask = 0ull;
                 if (MH) walk_mh<4>(a, v, e0 + (lane & 7u), e0 + len, 8, k, nvis);
@@ -1493,6 +1513,8 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
         if (gtid == 0) {  // bookkeeping: uncoloured at the start of round k (off the round top)
             if (k > 0) {
                 const int prv = (int)((k + 2) % 3);
+                // read and cleared in one atomic (performed before this block's
+                // next arrival; only gtid 0 reads these slots)
                 rem -= (int64_t)__ldcg(&a.ctr[cK + 16 * prv]);
                 a.ctr[cK + 16 * prv] = 0ull;  // only gtid 0 reads these slots
             }
@@ -1512,8 +1534,8 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
             }
         }
         schedule_fresh<JP>(a, prs, t_round);
-        stage_flush(a, prs, t_round);
-        if (!grid_barrier_rw(a, k, (int)((k + 1) % 3), stage().rd)) return;
+        stage_flush(a, prs, t_round, kRelax);
+        if (!grid_barrier_rw(a, k, (int)((k + 1) % 3), stage().rd, !kRelax)) return;
         if (PROF && gtid == 0) {
             const unsigned long long t = gtimer();
             if ((int64_t)k < a.nk_cap) a.rstat[16 * k + 4] = (int64_t)(t - t0);
@@ -1522,6 +1544,35 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
         }
     }
     (void)wpb;
+    if (kRelax) {
+        // one release / acquire barrier (every block's stamps and colours are
+        // visible), then each colour of round k >= 1 that was written as the
+        // max 2k becomes the min 2k+1 if v's lo side was freed second by
+        // round k (Zlo[v] <= k: min wins, Alg.5 L37-42, R9); a stamp of a
+        // later round never changes it.  The coloured vertices are counted
+        // here (the completion check).
+        __syncthreads();
+        if (threadIdx.x == 0) {
+            atom_add_release(a.ctr + cFin, 1ull);
+            const unsigned long long t0f = gtimer();
+            while (ld_acquire(a.ctr + cFin) < gridDim.x) {
+                if (gtimer() - t0f > 4000000000ull) {
+                    flag_error(a, 100, k, blockIdx.x);
+                    break;
+                }
+            }
+        }
+        __syncthreads();
+        uint32_t ncol = 0;
+        for (unsigned long long v = gtid; v < (unsigned long long)n; v += nthreads) {
+            const uint32_t c = __ldcg(a.C + v);
+            if (c == GC_UNC) continue;
+            ++ncol;
+            if ((c & 1u) == 0u && __ldcg(a.Zlo + v) <= (c >> 1)) a.C[v] = c | 1u;
+        }
+        const unsigned s = __reduce_add_sync(kFull, ncol);
+        if (lane == 0 && s) atomicAdd(&a.ctr[cCol], (unsigned long long)s);
+    }
     if (JP && a.jpv == 3) {
         // colours were round indices: C[v] <- colour of its round (the last
         // round's colour is this block's cprev; earlier ones are in cr)
@@ -1537,7 +1588,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
         a.ctr[cIters] = k;
         // the colourings of round k-1 (init's for k == 0) not yet subtracted
         rem -= (int64_t)__ldcg(&a.ctr[cK + 16 * (k == 0 ? 0 : (int)((k + 2) % 3))]);
-        a.ctr[cCol] = (unsigned long long)(n - rem);
+        if (!kRelax) a.ctr[cCol] = (unsigned long long)(n - rem);
         if (PROF) a.ctr[cPhaseNs + 1] = t_rounds;
     }
     if (PROF) {
