@@ -111,7 +111,15 @@ constexpr uint32_t kNever = 0xFFFFFFFFu;  // Z: side never free (yet)
 #ifndef GC_COUNT_THREADS
 #define GC_COUNT_THREADS 512
 #endif
-constexpr int kThreads = GC_COUNT_THREADS;  // one block per SM
+#ifndef GC_COUNT_THREADS_MAXMIN
+#define GC_COUNT_THREADS_MAXMIN 768  // measured on R-MAT s24 (max-min, relaxed rounds): 512 -> 18.9 ms,
+                                     // 768 -> 18.4, 896 -> 19.2, 1024 -> 19.3 (64 registers)
+#endif
+constexpr int kThreads = GC_COUNT_THREADS;  // one block per SM (JP, multi-hash: more registers)
+// threads per block of a kernel variant (max-min: 80 registers, no spills)
+template <bool JP, bool MH>
+constexpr int threads_for() { return (!JP && !MH) ? GC_COUNT_THREADS_MAXMIN : GC_COUNT_THREADS; }
+constexpr int kThreadsMax = GC_COUNT_THREADS_MAXMIN > GC_COUNT_THREADS ? GC_COUNT_THREADS_MAXMIN : GC_COUNT_THREADS;
 #ifndef GC_SHORT_MAX
 #define GC_SHORT_MAX 32
 #endif
@@ -398,7 +406,7 @@ struct Stage {
 #if GC_PACKED
     uint32_t htab[kHTab];           // hash set of the big vertices (kNone = empty)
 #endif
-    uint32_t wbits[kThreads / 32][32];  // JP: per-warp 1024-bit mex window
+    uint32_t wbits[kThreadsMax / 32][32];  // JP: per-warp 1024-bit mex window
     uint32_t cset[kCSetWords];          // Alg.4: the block's share of the round's colour set
     uint32_t cprev;                     // Alg.4: colour of the previous round
     unsigned cmin;                      // Alg.4: block reduction scratch
@@ -1204,7 +1212,7 @@ template <bool PROF, bool JP, bool MH>
 // __grid_constant__: helpers take `const CArgs &`; without it the reference
 // to a kernel parameter forces a per-thread local copy of CArgs (272 B of
 // stack, every field access an LDL through L1): 31.1 -> 28.7 ms on R-MAT s24.
-__global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_constant__ CArgs a) {
+__global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent(const __grid_constant__ CArgs a) {
     const unsigned lane = lane_id();
     const unsigned long long gtid = (unsigned long long)blockIdx.x * blockDim.x + threadIdx.x;
     const unsigned long long nthreads = (unsigned long long)gridDim.x * blockDim.x;
@@ -1513,8 +1521,6 @@ __global__ void __launch_bounds__(kThreads, 1) k_count_persistent(const __grid_c
         if (gtid == 0) {  // bookkeeping: uncoloured at the start of round k (off the round top)
             if (k > 0) {
                 const int prv = (int)((k + 2) % 3);
-                // read and cleared in one atomic (performed before this block's
-                // next arrival; only gtid 0 reads these slots)
                 rem -= (int64_t)__ldcg(&a.ctr[cK + 16 * prv]);
                 a.ctr[cK + 16 * prv] = 0ull;  // only gtid 0 reads these slots
             }
@@ -1853,7 +1859,7 @@ int launch(gc_graph *g, CArgs &a, int *blocks_out) {
     GC_CUDA_TRY(cudaFuncSetAttribute(k_count_persistent<PROF, JP, MH>,
                                      cudaFuncAttributeMaxDynamicSharedMemorySize, (int)kStageBytes));
     GC_CUDA_TRY(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_count_persistent<PROF, JP, MH>,
-                                                              kThreads, kStageBytes));
+                                                              threads_for<JP, MH>(), kStageBytes));
     if (per_sm < 1) {
         set_error("persistent count kernel cannot be resident");
         return GC_ERR_CUDA;
@@ -1899,7 +1905,7 @@ int launch(gc_graph *g, CArgs &a, int *blocks_out) {
     }
     cudaLaunchConfig_t cfg = {};
     cfg.gridDim = dim3(blocks);
-    cfg.blockDim = dim3(kThreads);
+    cfg.blockDim = dim3(threads_for<JP, MH>());
     cfg.dynamicSmemBytes = kStageBytes;
     cfg.stream = g->stream;
     cfg.attrs = attrs;
