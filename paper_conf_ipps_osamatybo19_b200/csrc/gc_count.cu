@@ -94,6 +94,13 @@ constexpr bool kSkipDead = GC_SKIP_DEAD != 0;
 constexpr bool kRelaxedArrive = GC_RELAXED_ARRIVE != 0;
 
 
+#ifndef GC_NO_PF_CI
+#define GC_NO_PF_CI 1  // 1: no L2 prefetch of the next round's short rows (measured: 18.33 vs 18.43 ms with it)
+#endif
+#ifndef GC_NO_PF_RO
+#define GC_NO_PF_RO 0  // experiments: no L2 prefetch of a freed vertex's row offsets
+#endif
+
 #ifndef GC_PACKED
 #define GC_PACKED 0  // 1: 32-bit (hi << 16 | lo) round counts -- max-min only (no JP / multi-hash branch);
                      // measured 27.9 vs 28.1 ms on R-MAT s24, not worth the restriction
@@ -633,8 +640,8 @@ __device__ __forceinline__ void schedule_rows(const CArgs &a, bool pred, uint32_
     it.lf = (uint32_t)len | ff;
     it.e0 = rs;
     if (shortrow && len > 0) {  // the row walked next round: HBM -> L2 now (<= 2 lines)
-        asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ci + rs));
-        asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ci + rs + len - 1));
+        if (!GC_NO_PF_CI) asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ci + rs));
+        if (!GC_NO_PF_CI) asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ci + rs + len - 1));
     }
     stage_append(a, shortrow, it, 0);
     unsigned lm = __ballot_sync(kFull, pred && !shortrow);
@@ -820,7 +827,7 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint64_t pv, in
 #else
             // its row offsets are loaded at the end of the round: start the
             // HBM -> L2 transfer now
-            asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ro + w[q]));
+            if (!GC_NO_PF_RO) asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ro + w[q]));
 #endif
             const unsigned pos = atomicAdd(&stage().nf, 1u);
             if (pos < (unsigned)kStF) {
@@ -1038,8 +1045,8 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
             it.lf = (uint32_t)len | fl;
             it.e0 = rs;
             if (len > 0) {  // the row walked next round: HBM -> L2 now (<= 2 lines)
-                asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ci + rs));
-                asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ci + re - 1));
+                if (!GC_NO_PF_CI) asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ci + rs));
+                if (!GC_NO_PF_CI) asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ci + re - 1));
             }
             const unsigned pos = atomicAdd(&st.n[0], 1u);
             if (pos < (unsigned)kStS) {
@@ -1261,8 +1268,26 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
     // N_0 = n (written here: a colouring whose round 0 walks no row ends
     // before the round loop's bookkeeping)
     if (gtid == 0 && a.nk_cap > 0) a.nk[0] = n;
-    // lane per vertex: a zero count colours v in round 0 (min wins, R9)
-    for (unsigned long long base = gwarp * 32; base < (unsigned long long)n; base += nwarps * 32) {
+    // lane per vertex: a zero count colours v in round 0 (min wins, R9).  The
+    // count word and the row offsets of kInitU batches of 32 vertices are
+    // loaded together up front (independent loads: the phase is a stream)
+    constexpr int kInitU = 4;
+    for (unsigned long long base0 = gwarp * 32 * kInitU; base0 < (unsigned long long)n;
+         base0 += nwarps * 32 * kInitU) {
+      unsigned long long cpre[kInitU];
+      int64_t rspre[kInitU], repre[kInitU];
+#pragma unroll
+      for (int b = 0; b < kInitU; ++b) {
+        const unsigned long long vv = base0 + 32ull * b + lane;
+        const bool ok = !MH && vv < (unsigned long long)n;
+        cpre[b] = ok ? __ldcs(a.cnt + vv) : 0x100000001ull;
+        rspre[b] = ok ? __ldg(a.ro + vv) : 0;
+        repre[b] = ok ? __ldg(a.ro + vv + 1) : 0;
+      }
+#pragma unroll
+      for (int b = 0; b < kInitU; ++b) {
+        const unsigned long long base = base0 + 32ull * b;
+        if (base >= (unsigned long long)n) break;
         const uint32_t v = (uint32_t)(base + lane);
         const bool valid = (int64_t)(base + lane) < n;
         uint32_t hi = 1u, lo = 1u, code = kNever;
@@ -1274,7 +1299,7 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
                 else if ((uint32_t)(c >> 32) == 0u) code = min(code, ((uint32_t)j << 1) | 1u);
             }
         } else {
-            const unsigned long long c = valid ? a.cnt[v] : 0x100000001ull;
+            const unsigned long long c = cpre[b];
             hi = (uint32_t)(c >> 32);
             lo = (uint32_t)c;
         }
@@ -1298,8 +1323,8 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
                 a.C[v] = zero ? (lo == 0u ? 1u : 0u) : GC_UNC;
             }
             if (zero) {
-                rs = a.ro[v];
-                re = a.ro[v + 1];
+                rs = MH ? a.ro[v] : rspre[b];
+                re = MH ? a.ro[v + 1] : repre[b];
             }
         }
         const unsigned word = __ballot_sync(kFull, zero);
@@ -1311,6 +1336,7 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
         if (lane == 0 && word) atomicAdd(&stage().colored, (unsigned)__popc(word));
         // walked in round 0 (the free side's flag: its neighbours, if any, are dead)
         schedule_rows<JP>(a, zero && re > rs, v, rs, re - rs, (!JP && !MH && lo == 0u) ? kLoSide : 0u);
+      }
     }
     stage_flush(a);
     if (!grid_barrier_rw(a, 0, 0, stage().rd)) return;
