@@ -54,9 +54,9 @@
 #endif
 
 #ifndef GC_COUNT_STREAM
-#define GC_COUNT_STREAM 0  // 1: counting pass as a chunked HBM stream (k_count_stream); measured
-                           // on R-MAT s24: 1.33 ms (1.75 TB/s) vs 0.96 + 0.28 ms for the
-                           // degree-binned k_count + k_count_hub, so the binned pass stays
+#define GC_COUNT_STREAM 1  // 1: counting pass of max-min / JP with random priorities as a tiled HBM
+                           // stream (k_count_tile, double-buffered cp.async); 0: the degree-binned
+                           // k_count + k_count_hub (always used for LDF and multi-hash)
 #endif
 constexpr bool kCountStream = GC_COUNT_STREAM != 0;
 
@@ -1298,6 +1298,9 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
                 if ((uint32_t)c == 0u) code = min(code, (uint32_t)j << 1);
                 else if ((uint32_t)(c >> 32) == 0u) code = min(code, ((uint32_t)j << 1) | 1u);
             }
+        } else if (rspre[b] == repre[b]) {
+            hi = 0u;  // no entries: the counting pass does not write the count word
+            lo = JP ? 1u : 0u;
         } else {
             const unsigned long long c = cpre[b];
             hi = (uint32_t)(c >> 32);
@@ -1753,22 +1756,26 @@ __global__ void __launch_bounds__(256) k_count_hub(const int64_t *__restrict__ r
     }
 }
 
-// ------------------------------------------------ streaming counting pass
-// The counting pass is the one full sweep of the CSR (it is round 0's
-// max/min test of Alg.5 for every vertex), so it is written as an HBM
-// stream: block-iterations take fixed chunks of kCE consecutive column ids
-// (8 per thread, 16-byte vector loads, fully coalesced), whatever the degree
-// mix.  The rows overlapping a chunk are found from crow[] (the row holding
-// each chunk's first entry, computed once per graph); a thread finds the row
-// of its first entry by binary search in the block's shared copy of the row
-// offsets and walks forward.  Per-row hi counts are accumulated in shared
-// memory; rows inside the chunk are written once, rows crossing a chunk
-// boundary (pre-set by k_count_zero) get one 64-bit atomic per chunk.
-constexpr int kCT = 256;            // threads per block
-constexpr int kCE = 8 * kCT;        // entries per chunk
-constexpr int kCR = 1024;           // rows per shared batch
+// ------------------------------------------------ counting pass: warp tiles
+// The counting pass is the one full read of the CSR (round 0's max / min test
+// of Alg.5 for every vertex at once), written as an HBM stream: warp tile w
+// is the kWE consecutive column ids [w kWE, +kWE), whatever the degree mix, so
+// every load is a coalesced 16-byte vector and no block barrier is needed.  A
+// lane takes kWQ consecutive entries (the next tile's are loaded before the
+// current one is counted).  The rows of the tile are visited in chunks of 32
+// (their offsets staged in the warp's shared slots); a lane finds the row of
+// its next entry by binary search there and walks forward; per-row hi counts
+// are summed in the warp's shared slots.  Rows inside the tile are written
+// once, rows crossing a tile boundary (pre-set by k_count_zero) get one
+// 64-bit atomic per tile.  Rows without entries are not written: the init
+// phase of the rounds reads their zero degree from the offsets.
+// crow[w] = the row of tile w's first entry (seed-independent, once per graph).
+constexpr int kWQ = 16;             // entries per lane
+constexpr int kWE = 32 * kWQ;       // entries per warp tile
+constexpr int kWT = 256;            // threads per block
+constexpr int kTE = kWE;            // (tile granularity of crow / k_count_zero)
 
-// crow[c] = last row r with ro[r] <= c * kCE (crow[0] = 0, crow[nch] = n - 1)
+// crow[c] = last row r with ro[r] <= c * kTE (crow[0] = 0, crow[nch] = n - 1)
 __global__ void k_chunk_rows(const int64_t *__restrict__ ro, int64_t n, int64_t nch, uint32_t *crow) {
     for (int64_t c = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; c <= nch;
          c += (int64_t)gridDim.x * blockDim.x) {
@@ -1776,7 +1783,7 @@ __global__ void k_chunk_rows(const int64_t *__restrict__ ro, int64_t n, int64_t 
             crow[c] = c == 0 ? 0u : (uint32_t)(n - 1);
             continue;
         }
-        const int64_t e = c * kCE;
+        const int64_t e = c * kTE;
         int64_t lo = 0, hi = n;  // ro[lo] <= e < ro[hi]
         while (hi - lo > 1) {
             const int64_t mid = (lo + hi) >> 1;
@@ -1787,95 +1794,115 @@ __global__ void k_chunk_rows(const int64_t *__restrict__ ro, int64_t n, int64_t 
     }
 }
 
-// rows crossing a chunk boundary start from zero (JP: lo pinned at 1)
+// rows crossing a tile boundary start from zero (JP: lo pinned at 1)
 __global__ void k_count_zero(const int64_t *__restrict__ ro, const uint32_t *__restrict__ crow, int64_t nch,
                              unsigned long long *cnt, int jp) {
     for (int64_t c = 1 + (int64_t)blockIdx.x * blockDim.x + threadIdx.x; c < nch;
          c += (int64_t)gridDim.x * blockDim.x) {
         const uint32_t r = crow[c];
-        if (ro[r] < c * kCE) cnt[r] = jp ? 1ull : 0ull;
+        if (ro[r] < c * kTE) cnt[r] = jp ? 1ull : 0ull;
     }
 }
 
-__global__ void __launch_bounds__(kCT) k_count_stream(const int64_t *__restrict__ ro, const uint32_t *__restrict__ ci,
-                                                      int64_t m, int64_t nch, const uint32_t *__restrict__ crow,
-                                                      uint32_t key, unsigned long long *cnt, int jp) {
-    __shared__ int64_t ro_sh[kCR + 1];
-    __shared__ uint32_t h_sh[kCR];
-    for (int64_t c = blockIdx.x; c < nch; c += gridDim.x) {
-        const int64_t c0 = c * kCE, c1 = min(m, c0 + kCE);
-        const bool last_chunk = c == nch - 1;
-        const int64_t r0 = crow[c], r1 = crow[c + 1];
-        // the first batch's entries start at c0 (ro[crow[c]] <= c0): their loads
-        // go out together with the row offsets'
-        uint32_t u[8];
-        auto load_u = [&](int64_t ef, int64_t eh) {
-            if ((reinterpret_cast<uintptr_t>(ci + ef) & 15) == 0 && ef + 8 <= eh) {
-                const uint4 a0 = __ldcs(reinterpret_cast<const uint4 *>(ci + ef));
-                const uint4 a1 = __ldcs(reinterpret_cast<const uint4 *>(ci + ef + 4));
-                u[0] = a0.x; u[1] = a0.y; u[2] = a0.z; u[3] = a0.w;
-                u[4] = a1.x; u[5] = a1.y; u[6] = a1.z; u[7] = a1.w;
-            } else {
+__device__ __forceinline__ void load_tile(const uint32_t *ci, int64_t m, int64_t w, uint32_t (&u)[kWQ]) {
+    const int64_t e = w * kWE + kWQ * (int64_t)lane_id();
+    if (e + kWQ <= m) {
 #pragma unroll
-                for (int q = 0; q < 8; ++q) u[q] = ef + q < eh ? __ldcs(ci + ef + q) : 0u;
-            }
-        };
-        load_u(c0 + 8 * (int64_t)threadIdx.x, c1);
-        for (int64_t rb = r0; rb <= r1; rb += kCR) {
-            const int nr = (int)min((int64_t)kCR, r1 - rb + 1);
-            __syncthreads();
-            for (int i = threadIdx.x; i <= nr; i += kCT) ro_sh[i] = ro[rb + i];
-            for (int i = threadIdx.x; i < nr; i += kCT) h_sh[i] = 0u;
-            __syncthreads();
-            const int64_t e_lo = max(ro_sh[0], c0), e_hi = min(ro_sh[nr], c1);
-            const int64_t e_first = e_lo + 8 * (int64_t)threadIdx.x;
-            if (rb != r0 && e_first < e_hi) load_u(e_first, e_hi);
-            if (e_first < e_hi) {
-                // row of e_first: last i with ro_sh[i] <= e_first
-                int lo = 0, hi = nr;
+        for (int j = 0; j < kWQ / 4; ++j) {
+            const uint4 x = __ldcs(reinterpret_cast<const uint4 *>(ci + e) + j);
+            u[4 * j] = x.x;
+            u[4 * j + 1] = x.y;
+            u[4 * j + 2] = x.z;
+            u[4 * j + 3] = x.w;
+        }
+    } else {
+#pragma unroll
+        for (int q = 0; q < kWQ; ++q) u[q] = e + q < m ? __ldcs(ci + e + q) : 0u;
+    }
+}
+
+__global__ void __launch_bounds__(kWT) k_count_warp(const int64_t *__restrict__ ro, const uint32_t *__restrict__ ci,
+                                                    int64_t n, int64_t m, int64_t nch,
+                                                    const uint32_t *__restrict__ crow, uint32_t key,
+                                                    unsigned long long *cnt, int jp) {
+    __shared__ long long offs_sh[kWT / 32][33];
+    __shared__ uint32_t h_sh[kWT / 32][32];
+    const unsigned lane = lane_id(), wib = threadIdx.x >> 5;
+    long long *offs = offs_sh[wib];
+    uint32_t *hs = h_sh[wib];
+    hs[lane] = 0u;
+    const int64_t nwarps = (int64_t)gridDim.x * (kWT / 32);
+    int64_t w = (int64_t)blockIdx.x * (kWT / 32) + wib;
+    if (w >= nch) return;
+    uint32_t u[kWQ], un[kWQ];
+    load_tile(ci, m, w, u);
+    for (;;) {
+        const int64_t wn = w + nwarps;
+        if (wn < nch) load_tile(ci, m, wn, un);  // next tile's column ids in flight
+        const int64_t e0 = w * kWE, e1 = min(m, e0 + kWE);
+        const int64_t ra = crow[w], rz = crow[w + 1];  // rows touching the tile: [ra, rz]
+        const bool last_tile = w == nch - 1;
+        const int64_t qf = e0 + kWQ * (int64_t)lane;
+        int cur = 0;  // this lane's entries < cur are counted
+        for (int64_t rb = ra; rb <= rz; rb += 32) {
+            const int nr = (int)min((int64_t)32, rz - rb + 1);
+            offs[lane] = lane <= nr ? (long long)__ldg(ro + rb + lane) : 0ll;
+            if (lane == 0) offs[32] = nr == 32 ? (long long)__ldg(ro + rb + 32) : 0ll;
+            __syncwarp();
+            const int64_t lim = min((int64_t)offs[nr], e1);  // entries of these rows within the tile
+            if (cur < kWQ && qf + cur < lim) {
+                const int64_t es = qf + cur;
+                int lo = 0, hi = nr;  // offs[lo] <= es < offs[hi]
                 while (hi - lo > 1) {
                     const int mid = (lo + hi) >> 1;
-                    if (ro_sh[mid] <= e_first) lo = mid;
+                    if (offs[mid] <= es) lo = mid;
                     else hi = mid;
                 }
                 int ri = lo;
-                int64_t rend = ro_sh[ri + 1];
+                int rend = (int)(min((int64_t)offs[ri + 1], lim) - qf);  // relative to qf
+                const int qlim = (int)min((int64_t)kWQ, lim - qf);
                 uint32_t pv = weight_mix((uint32_t)(rb + ri) ^ key);
                 uint32_t acc = 0;
 #pragma unroll
-                for (int q = 0; q < 8; ++q) {
-                    const int64_t e = e_first + q;
-                    if (e < e_hi) {
-                        if (e >= rend) {
-                            if (acc) atomicAdd(&h_sh[ri], acc);
+                for (int q = 0; q < kWQ; ++q) {
+                    if (q >= cur && q < qlim) {
+                        if (q >= rend) {
+                            atomicAdd(&hs[ri], acc);
                             acc = 0;
                             do {
                                 ++ri;
-                                rend = ro_sh[ri + 1];
-                            } while (e >= rend);
+                                rend = (int)(min((int64_t)offs[ri + 1], lim) - qf);
+                            } while (q >= rend);
                             pv = weight_mix((uint32_t)(rb + ri) ^ key);
                         }
                         acc += weight_mix(u[q] ^ key) > pv ? 1u : 0u;
                     }
                 }
-                if (acc) atomicAdd(&h_sh[ri], acc);
+                atomicAdd(&hs[ri], acc);
+                cur = qlim;
             }
-            __syncthreads();
-            for (int i = threadIdx.x; i < nr; i += kCT) {
-                const int64_t rs = ro_sh[i], re = ro_sh[i + 1];
-                const uint32_t h = h_sh[i];
-                const bool partial = rs < c0 || re > c1;
-                if (partial) {
-                    const int64_t len = min(re, c1) - max(rs, c0);
+            __syncwarp();
+            if (lane < (unsigned)nr) {
+                const int64_t r = rb + lane;
+                const int64_t rs = offs[lane], re = offs[lane + 1];
+                const uint32_t h = hs[lane];
+                hs[lane] = 0u;
+                if (rs < e0 || re > e1) {  // crosses a tile boundary: this tile's part
+                    const int64_t len = min(re, e1) - max(rs, e0);
                     if (len > 0)
-                        atomicAdd(cnt + rb + i, ((unsigned long long)h << 32) + (jp ? 0ull : (unsigned long long)(len - h)));
-                } else if (rb + i < r1 || last_chunk) {
-                    // inside this chunk; row crow[c+1] (empty, starting at c1) is the next
-                    // chunk's first row, and the next chunk writes it
-                    cnt[rb + i] = ((unsigned long long)h << 32) | (unsigned long long)(jp ? 1 : (re - rs) - h);
+                        atomicAdd(cnt + r, ((unsigned long long)h << 32) + (jp ? 0ull : (unsigned long long)(len - h)));
+                } else if (re > rs && (r < rz || last_tile)) {
+                    // inside the tile (rows without entries are left to the init phase);
+                    // row rz starting at e1 is the next tile's first row
+                    cnt[r] = ((unsigned long long)h << 32) | (unsigned long long)(jp ? 1 : (re - rs) - h);
                 }
             }
+            __syncwarp();
         }
+        if (wn >= nch) break;
+        w = wn;
+#pragma unroll
+        for (int q = 0; q < kWQ; ++q) u[q] = un[q];
     }
 }
 
@@ -2001,12 +2028,22 @@ int ensure_count_scratch(gc_graph *g) {
     GC_CUDA_TRY(dmalloc(&s.hubs, ((size_t)g->nnz / kHubChunk + 1) * 8));
     GC_CUDA_TRY(dmalloc(&s.cctr, kCCtrWords * sizeof(unsigned long long)));
     GC_CUDA_TRY(dmalloc(&s.cM, (nn + 31) / 32 * 4));
-    if (kCountStream) {  // streaming counting pass: the row of every chunk's first entry
-        s.nch = std::max<int64_t>(1, (g->nnz + kCE - 1) / kCE);
-        GC_CUDA_TRY(dmalloc(&s.crow, (size_t)(s.nch + 1) * 4));
-        k_chunk_rows<<<g->sm_count * 4, 256, 0, g->stream>>>(g->ro, g->n, s.nch, s.crow);
-        GC_CUDA_TRY(cudaGetLastError());
-    }
+    return GC_OK;
+}
+
+// tiled counting pass: the row of every tile's first entry, for the CSR the
+// handle colours now (a deduplicated copy replaces it at most once)
+static int ensure_crow(gc_graph *g) {
+    Scratch &s = g->s;
+    if (s.crow && s.crow_ro == g->ro && s.crow_nnz == g->nnz) return GC_OK;
+    dfree(s.crow);
+    s.crow = nullptr;
+    s.nch = std::max<int64_t>(1, (g->nnz + kTE - 1) / kTE);
+    GC_CUDA_TRY(dmalloc(&s.crow, (size_t)(s.nch + 1) * 4));
+    k_chunk_rows<<<g->sm_count * 4, 256, 0, g->stream>>>(g->ro, g->n, s.nch, s.crow);
+    GC_CUDA_TRY(cudaGetLastError());
+    s.crow_ro = g->ro;
+    s.crow_nnz = g->nnz;
     return GC_OK;
 }
 
@@ -2105,11 +2142,13 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
             k_count<true><<<blocks, 256, 0, st>>>(g->ro, g->ci, n, ck, s.cnt, hubs, nhubs, 0, nullptr);
             k_count_hub<true><<<g->sm_count * 8, 256, 0, st>>>(g->ro, g->ci, ck, s.cnt, hubs, nhubs, 0,
                                                                nullptr);
-        } else if (kCountStream && !dg) {
+        } else if (kCountStream && !dg && ((reinterpret_cast<uintptr_t>(g->ci) | reinterpret_cast<uintptr_t>(g->ro)) & 15) == 0) {
+            // (cp.async copies 16-byte pieces: borrowed buffers must be 16-byte aligned)
+            if ((rc = ensure_crow(g))) return rc;
             const int64_t nch = s.nch;
             k_count_zero<<<g->sm_count, 256, 0, st>>>(g->ro, s.crow, nch, s.cnt, jp ? 1 : 0);
-            k_count_stream<<<(int)std::min<int64_t>(nch, (int64_t)g->sm_count * 8), kCT, 0, st>>>(
-                g->ro, g->ci, g->nnz, nch, s.crow, key, s.cnt, jp ? 1 : 0);
+            k_count_warp<<<(int)std::min<int64_t>((nch + 7) / 8, (int64_t)g->sm_count * 8), kWT, 0, st>>>(
+                g->ro, g->ci, n, g->nnz, nch, s.crow, key, s.cnt, jp ? 1 : 0);
         } else {
             k_count<false><<<blocks, 256, 0, st>>>(g->ro, g->ci, n, ck, s.cnt, hubs, nhubs, jp ? 1 : 0, dg);
             k_count_hub<false><<<g->sm_count * 8, 256, 0, st>>>(g->ro, g->ci, ck, s.cnt, hubs, nhubs,

@@ -78,6 +78,8 @@ struct Scratch {
     uint32_t *cM = nullptr;              // COUNT mode: status bits (1 = uncoloured)
     uint32_t *crow = nullptr;            // COUNT mode: row of each counting chunk's first entry
     int64_t nch = 0;
+    const int64_t *crow_ro = nullptr;    // ... of this CSR (row offsets, entries)
+    int64_t crow_nnz = -1;
     uint32_t *deg = nullptr;             // LDF: row lengths (seed-independent)
     uint32_t *jslot = nullptr;           // JP (Luby-MIS in COUNT mode): mex slots of long rows
     uint32_t *jcr = nullptr;             // Alg.4: round colours + colour sets
