@@ -101,6 +101,12 @@ constexpr bool kRelaxedArrive = GC_RELAXED_ARRIVE != 0;
 #define GC_NO_PF_RO 0  // experiments: no L2 prefetch of a freed vertex's row offsets
 #endif
 
+#ifndef GC_EAGER_FRESH
+#define GC_EAGER_FRESH 0  // 1: max-min walks schedule the vertices they free right away (warp-level);
+                          // measured 20.83 vs 18.10 ms on R-MAT s24: loads issued behind the round's atomics wait
+#endif
+constexpr bool kEagerFresh = GC_EAGER_FRESH != 0;
+
 #ifndef GC_PACKED
 #define GC_PACKED 0  // 1: 32-bit (hi << 16 | lo) round counts -- max-min only (no JP / multi-hash branch);
                      // measured 27.9 vs 28.1 ms on R-MAT s24, not worth the restriction
@@ -813,6 +819,22 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint64_t pv, in
                 flag_error(a, 4, k, w[q]);  // count underflow: adjacency not symmetric
             }
         }
+    }
+    if (!JP && kEagerFresh) {
+        // max-min: the warp schedules the neighbours it freed itself, right
+        // after its unit (their row offsets loaded together), so the block
+        // has no separate fresh step at the end of the round
+        int64_t rsq[Q], req[Q];
+#pragma unroll
+        for (int q = 0; q < Q; ++q) {
+            rsq[q] = fresh[q] ? __ldg(a.ro + w[q]) : 0;
+            req[q] = fresh[q] ? __ldg(a.ro + w[q] + 1) : 0;
+        }
+#pragma unroll
+        for (int q = 0; q < Q; ++q)
+            if (__any_sync(kFull, fresh[q]))
+                schedule_rows_slow<JP>(a, fresh[q], w[q], rsq[q], req[q] - rsq[q], kFirst | (hi[q] ? 0u : kLoSide));
+        return;
     }
     // (rare) newly scheduled neighbours go to the block's fresh list; their
     // rows are fetched once per block at the end of the round (schedule_fresh)
@@ -1568,7 +1590,7 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
                 }
             }
         }
-        schedule_fresh<JP>(a, prs, t_round);
+        if (!(kEagerFresh && !JP && !MH)) schedule_fresh<JP>(a, prs, t_round);
         stage_flush(a, prs, t_round, kRelax);
         if (!grid_barrier_rw(a, k, (int)((k + 1) % 3), stage().rd, !kRelax)) return;
         if (PROF && gtid == 0) {
@@ -1843,6 +1865,9 @@ __global__ void __launch_bounds__(kWT) k_count_warp(const int64_t *__restrict__ 
         const int64_t ra = crow[w], rz = crow[w + 1];  // rows touching the tile: [ra, rz]
         const bool last_tile = w == nch - 1;
         const int64_t qf = e0 + kWQ * (int64_t)lane;
+        uint32_t mx[kWQ];  // the entries' priorities
+#pragma unroll
+        for (int q = 0; q < kWQ; ++q) mx[q] = weight_mix(u[q] ^ key);
         int cur = 0;  // this lane's entries < cur are counted
         for (int64_t rb = ra; rb <= rz; rb += 32) {
             const int nr = (int)min((int64_t)32, rz - rb + 1);
@@ -1850,7 +1875,13 @@ __global__ void __launch_bounds__(kWT) k_count_warp(const int64_t *__restrict__ 
             if (lane == 0) offs[32] = nr == 32 ? (long long)__ldg(ro + rb + 32) : 0ll;
             __syncwarp();
             const int64_t lim = min((int64_t)offs[nr], e1);  // entries of these rows within the tile
-            if (cur < kWQ && qf + cur < lim) {
+            // this lane's entries [cur, qlim) of these rows, one row per step:
+            // the row's hi count = popcount of the entries whose priority beats
+            // the row vertex's (a 16-bit mask, no per-entry branches)
+            const int qlim = (int)max((int64_t)cur, min((int64_t)kWQ, lim - qf));
+            bool act = cur < qlim;
+            int ri = 0;
+            if (act) {
                 const int64_t es = qf + cur;
                 int lo = 0, hi = nr;  // offs[lo] <= es < offs[hi]
                 while (hi - lo > 1) {
@@ -1858,29 +1889,29 @@ __global__ void __launch_bounds__(kWT) k_count_warp(const int64_t *__restrict__ 
                     if (offs[mid] <= es) lo = mid;
                     else hi = mid;
                 }
-                int ri = lo;
-                int rend = (int)(min((int64_t)offs[ri + 1], lim) - qf);  // relative to qf
-                const int qlim = (int)min((int64_t)kWQ, lim - qf);
-                uint32_t pv = weight_mix((uint32_t)(rb + ri) ^ key);
-                uint32_t acc = 0;
+                ri = lo;
+            }
+            int qs = cur;
+            while (__any_sync(kFull, act)) {
+                if (act) {
+                    const int re_rel = (int)min((int64_t)offs[ri + 1] - qf, (int64_t)qlim);  // > qs
+                    const uint32_t pv = weight_mix((uint32_t)(rb + ri) ^ key);
+                    uint32_t g = 0;
 #pragma unroll
-                for (int q = 0; q < kWQ; ++q) {
-                    if (q >= cur && q < qlim) {
-                        if (q >= rend) {
-                            atomicAdd(&hs[ri], acc);
-                            acc = 0;
-                            do {
-                                ++ri;
-                                rend = (int)(min((int64_t)offs[ri + 1], lim) - qf);
-                            } while (q >= rend);
-                            pv = weight_mix((uint32_t)(rb + ri) ^ key);
-                        }
-                        acc += weight_mix(u[q] ^ key) > pv ? 1u : 0u;
+                    for (int q = 0; q < kWQ; ++q) g |= (mx[q] > pv ? 1u : 0u) << q;
+                    const uint32_t rng = ((1u << re_rel) - 1u) & ~((1u << qs) - 1u);
+                    const uint32_t hcount = (uint32_t)__popc(g & rng);
+                    if (hcount) atomicAdd(&hs[ri], hcount);
+                    qs = re_rel;
+                    act = qs < qlim;
+                    if (act) {  // the next row with entries here (skip empty rows)
+                        do {
+                            ++ri;
+                        } while (offs[ri + 1] - qf <= qs);
                     }
                 }
-                atomicAdd(&hs[ri], acc);
-                cur = qlim;
             }
+            cur = qlim;
             __syncwarp();
             if (lane < (unsigned)nr) {
                 const int64_t r = rb + lane;
