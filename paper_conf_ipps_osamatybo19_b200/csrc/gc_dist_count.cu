@@ -436,9 +436,13 @@ __device__ __forceinline__ void push_sk(const DCArgs &a, uint32_t val, uint32_t 
     if (at < (unsigned long long)a.n_loc) a.S[(int64_t)lst * a.n_loc + (int64_t)at] = val;
     else flag(a, 2, val);
 }
+// skip (DESIGN 7.0, dead side): the parity of v's colour names a side of v
+// that was free at the start of round k (odd: lo, all smaller neighbours are
+// coloured; even: hi, all larger ones), so decrements to that side's
+// neighbours are dead and not issued (skip 1: entries below v, 0: above)
 template <bool GHOST>
 __device__ __forceinline__ void walk_entries_k(const DCArgs &a, uint32_t pv, int64_t s, int64_t e, int64_t sub,
-                                               int64_t width, uint32_t k) {
+                                               int64_t width, uint32_t k, int skip) {
     for (int64_t i0 = s + sub; i0 < e; i0 += kQ * width) {
         uint32_t lw[kQ], wg[kQ];
         bool live[kQ];
@@ -460,6 +464,7 @@ __device__ __forceinline__ void walk_entries_k(const DCArgs &a, uint32_t pv, int
 #pragma unroll
         for (int q = 0; q < kQ; ++q) {
             hi[q] = pv > weight_mix(wg[q] ^ a.key);
+            live[q] = live[q] && hi[q] != (skip == 1);
             old[q] = live[q] ? atomicAdd(a.cnt + lw[q], hi[q] ? kDecHi : kDecLo) : 2ull;
         }
 #pragma unroll
@@ -508,8 +513,9 @@ __device__ __forceinline__ void walk_chunks(const DCArgs &a, bool ghost, unsigne
         const ChunkItem c = lc[i];
         const uint32_t pv = weight_mix(c.v ^ a.key);
         const int64_t c1 = c.c0 + (c.len & ~kGhostBit);
-        if (c.len & kGhostBit) walk_entries_k<true>(a, pv, c.c0, c1, threadIdx.x, blockDim.x, k);
-        else walk_entries_k<false>(a, pv, c.c0, c1, threadIdx.x, blockDim.x, k);
+        const int skip = (int)(__ldcg(a.C + c.v) & 1u);  // (written before the group barrier)
+        if (c.len & kGhostBit) walk_entries_k<true>(a, pv, c.c0, c1, threadIdx.x, blockDim.x, k, skip);
+        else walk_entries_k<false>(a, pv, c.c0, c1, threadIdx.x, blockDim.x, k, skip);
     }
 }
 
@@ -562,7 +568,9 @@ __global__ void __launch_bounds__(256) k_dc_persistent(const __grid_constant__ D
                 }
                 if (re - rs > kPLongMin) push_long_k(a, rs, re, vg, 0u, par);
             }
-            if (re - rs <= kPLongMin) walk_entries_k<false>(a, weight_mix(vg ^ a.key), rs, re, sub, 8, k);
+            if (re - rs <= kPLongMin)
+                walk_entries_k<false>(a, weight_mix(vg ^ a.key), rs, re, sub, 8, k,
+                                      ((it & kLoF) || a.Z[lv] <= k) ? 1 : 0);
         }
         // B. publish
         if (tl) atomicMax(tl + 0, gtimer_dp() - t_round);  // own walks done
@@ -661,7 +669,8 @@ __global__ void __launch_bounds__(256) k_dc_persistent(const __grid_constant__ D
                     a.C[pr.x] = pr.y;
                     if (ge - gs > kPLongMin) push_long_k(a, gs, ge, pr.x, 1u, par);
                 }
-                if (ge - gs <= kPLongMin) walk_entries_k<true>(a, weight_mix(pr.x ^ a.key), gs, ge, sub, 8, k);
+                if (ge - gs <= kPLongMin)
+                    walk_entries_k<true>(a, weight_mix(pr.x ^ a.key), gs, ge, sub, 8, k, (int)(pr.y & 1u));
             }
         }
         if (tl) atomicMax(tl + 3, gtimer_dp() - t_round);  // ghost walks done
