@@ -133,7 +133,7 @@ def source_sha(kernel: str) -> str:
     """sha256 (16 hex) of the CUDA source that defines `kernel` (the key that
     keeps a committed ncu capture from outliving a kernel change)."""
     import hashlib
-    src = {"k_count_persistent": "gc_count.cu", "k_count + k_count_hub": "gc_count.cu"}.get(kernel)
+    src = {"k_count_persistent": "gc_count.cu", "counting pass": "gc_count.cu"}.get(kernel)
     if src is None:
         return ""
     with open(os.path.join(ROOT, "paper_conf_ipps_osamatybo19_b200", "csrc", src), "rb") as f:
@@ -344,7 +344,9 @@ def main():
     # timed steps (libgc brackets the counting pass and the persistent kernel
     # with events on every colouring) and their algorithmic bytes per launch
     # (DESIGN.md 10): counting pass 16 n + 4 m; persistent kernel
-    # 16 n + 56 s + 32 ceil(m / 256) + 20 m, s = non-isolated vertices
+    # 16 n + 56 s + 32 ceil(m / 128) + 4 m + 16 A, s = non-isolated vertices,
+    # A = count decrements the kernel issued (gc_stats.visits: the walks skip
+    # neighbours on the walked vertex's free side)
     roof = None
     peak, peak_src = measured_peaks()
     if st.mode_used == gcb.MODE_COUNT and not use_dist and args.variant == "maxmin":
@@ -352,8 +354,9 @@ def main():
         s_nz = int((deg > 0).sum())
         m = nnz_global
         classes = {}
-        for c, name, nbytes in ((0, "k_count_persistent", 16 * n + 56 * s_nz + 32 * ((m + 255) // 256) + 20 * m),
-                                (1, "k_count + k_count_hub", 16 * n + 4 * m)):
+        A = int(st.visits)
+        for c, name, nbytes in ((0, "k_count_persistent", 16 * n + 56 * s_nz + 32 * ((m + 127) // 128) + 4 * m + 16 * A),
+                                (1, "counting pass", 16 * n + 4 * m)):
             t_ms = statistics.median(kms[c])
             ach = nbytes / 1e9 / (t_ms / 1e3)
             classes[name] = {"bound": "hbm", "achieved": ach, "peak": peak, "unit": "GB/s",
@@ -361,6 +364,8 @@ def main():
                              "launch_ms_median": t_ms, "bytes_per_launch": nbytes,
                              "launches_per_step": 1 if c == 0 else 2,
                              "share_of_step": t_ms / statistics.median(step_ms)}
+        classes["k_count_persistent"]["count_decrements"] = A
+        classes["k_count_persistent"]["bytes_formula"] = "16 n + 56 s + 32 ceil(m/128) + 4 m + 16 A"
         dom = classes["k_count_persistent"]
         roof = dict(dom)
         roof.update({"kernel": "k_count_persistent", "peak_source": peak_src,
@@ -381,7 +386,7 @@ def main():
                  gcb.MODE_EVENT_MULTI: {0: "k_eval", 1: "k_eval_big", 2: "k_notify",
                                         3: "k_notify_big"},
                  gcb.MODE_SWEEP: {0: "k_sweep", 1: "k_hub", 2: "other", 3: "other"},
-                 gcb.MODE_COUNT: {0: "k_count_persistent", 1: "k_count + k_count_hub",
+                 gcb.MODE_COUNT: {0: "k_count_persistent", 1: "counting pass",
                                   2: "init phase (round 0)", 3: "rounds"}}[sp.mode_used]
         if args.variant == "hash":
             names = {0: "k_hash_propose", 1: "k_hash_resolve", 2: "k_hash_table",

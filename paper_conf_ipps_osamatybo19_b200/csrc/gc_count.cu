@@ -1566,9 +1566,9 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
         if (PROF) {
             const unsigned s = __reduce_add_sync(kFull, nvis);
             if (lane == 0 && s) atomicAdd(&stage().vis, s);
-            nvis_tot += nvis;
-            nvis = 0;
         }
+        nvis_tot += nvis;  // (always: the count decrements issued, for the algorithmic bytes)
+        nvis = 0;
         if (gtid == 0) {  // bookkeeping: uncoloured at the start of round k (off the round top)
             if (k > 0) {
                 const int prv = (int)((k + 2) % 3);
@@ -1648,7 +1648,7 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
         if (!kRelax) a.ctr[cCol] = (unsigned long long)(n - rem);
         if (PROF) a.ctr[cPhaseNs + 1] = t_rounds;
     }
-    if (PROF) {
+    {
         const unsigned long long s = __reduce_add_sync(kFull, (unsigned)nvis_tot);
         if (lane == 0 && s) atomicAdd(&a.ctr[cVis], s);
     }
@@ -2285,6 +2285,7 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
         p.prof->launch_us.push_back(1e3f * (ms_all - ms_cnt));
         p.prof->ms[1] += ms_cnt;
         p.prof->launches[1] += 2;
+        if (!prof) p.prof->visits += (int64_t)h[cVis];  // count decrements issued (always counted)
     }
     if (prof) {
         p.prof->ms[2] += (double)h[cPhaseNs] / 1e6;

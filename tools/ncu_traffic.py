@@ -32,7 +32,8 @@ def main():
     for r in rows[2:]:
         name = r[ki]
         c = ("k_count_persistent" if "k_count_persistent" in name else
-             "k_count + k_count_hub" if ("k_count<" in name or "k_count_hub<" in name) else None)
+             "counting pass" if any(x in name for x in ("k_count<", "k_count_hub<", "k_count_warp", "k_count_zero"))
+             else None)
         if c is None:
             continue
         b = float(r[rd]) * scale[units[rd]] + float(r[wr]) * scale[units[wr]]
