@@ -107,6 +107,12 @@ constexpr bool kRelaxedArrive = GC_RELAXED_ARRIVE != 0;
 #endif
 constexpr bool kEagerFresh = GC_EAGER_FRESH != 0;
 
+#ifndef GC_DIRECT_FLUSH
+#define GC_DIRECT_FLUSH 1  // 1: max-min rounds reserve the next round's items right after the fresh
+                           // vertices' row offsets are in, then write them straight to the lists
+#endif
+constexpr bool kDirectFlush = GC_DIRECT_FLUSH != 0;
+
 #ifndef GC_PACKED
 #define GC_PACKED 0  // 1: 32-bit (hi << 16 | lo) round counts -- max-min only (no JP / multi-hash branch);
                      // measured 27.9 vs 28.1 ms on R-MAT s24, not worth the restriction
@@ -413,6 +419,9 @@ struct Stage {
     Item s[kStS];
     Item w[kStW];
     uint2 fresh[kStF];              // (w, lo side?) this block scheduled in the round
+    int64_t frs[kStF];              // direct flush: their row starts ...
+    uint2 fmeta[kStF];              // ... (row length, first slot among the block's direct items)
+    unsigned nd[2];                 // direct flush: the block's direct SL items / WL segments
 #if GC_EAGER_RO
     longlong2 fro[kStF];            // their row offsets (loaded by the freeing lane)
 #endif
@@ -616,6 +625,107 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
     if (threadIdx.x < 2) st.n[threadIdx.x] = 0;
     if (prs && threadIdx.x == 0)
         red_max(prs + 8, gtimer() - t_round);
+}
+
+// Whole block, end of a max-min round (relaxed rounds, kDirectFlush): one
+// thread per fresh vertex loads its row offsets and takes its slots among
+// the block's items of the next round (an SL item, or its WL segments); the
+// block then reserves them with its arrival (one relaxed atomic on the round
+// word) and writes every item straight to its slot -- long rows expanded by
+// a warp each -- while the barrier completes (the items carry round tags the
+// consumers check).  Items staged in shared memory by the rare overflow
+// paths of the walks go first.
+__device__ __forceinline__ void fresh_flush_direct(const CArgs &a) {
+    Stage &st = stage();
+    __syncthreads();  // the units are done
+    const unsigned nf = min(st.nf, (unsigned)kStF);
+    for (unsigned t = threadIdx.x; t < nf; t += blockDim.x) {
+        const uint2 f = st.fresh[t];
+        const int64_t rs = a.ro[f.x], re = a.ro[f.x + 1];
+        const int64_t len = re - rs;
+        unsigned pos;
+        if (len <= kShortMax) {
+            pos = atomicAdd(&st.nd[0], 1u);
+            if (!GC_NO_PF_CI && len > 0) asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ci + rs));
+        } else {
+            pos = atomicAdd(&st.nd[1], (unsigned)((len + kSeg - 1) / kSeg));
+        }
+        st.frs[t] = rs;
+        st.fmeta[t] = make_uint2((uint32_t)len, pos);
+    }
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        const unsigned c0 = min(st.n[0], (unsigned)kStS), c1 = min(st.n[1], (unsigned)kStW);
+        const unsigned long long t0 = c0 + st.nd[0], t1 = c1 + st.nd[1];
+        if (st.colored) atom_add_global(st.ccol, (unsigned long long)st.colored);
+        st.colored = 0;
+        // the reservation of both lists is the barrier arrival (relaxed: 7.0)
+        const unsigned long long rv = atom_add_global(st.rw, rw_add(t0, 0) + rw_add(t1, 1) + kRwArr);
+        const unsigned long long r0 = rw_field(rv, 0), r1 = rw_field(rv, 1);
+        if (r0 + t0 > kMSL || r1 + t1 > kMWL) flag_error(a, 9, 0, 0);  // a round word field overflowed
+        st.base[0] = st.nbase[0] + r0;
+        st.base[1] = st.nbase[1] + r1;
+        st.n[0] = c0;
+        st.n[1] = c1;
+        if (st.base[0] + t0 > a.sl_cap || st.base[1] + t1 > a.wl_cap) {
+            flag_error(a, 2, 0, 0);
+            st.n[0] = st.n[1] = 0;
+            st.nf = 0;
+        }
+        st.nlong = 0;
+    }
+    __syncthreads();
+    Item *const sl = a.SL + grp_base(a, 0), *const wl = a.WL + grp_base(a, 1);
+    const unsigned c0 = st.n[0], c1 = st.n[1];
+    const unsigned long long b0 = st.base[0], b1 = st.base[1];
+    for (unsigned i = threadIdx.x; i < c0; i += blockDim.x) gput(sl + b0 + i, st.s[i]);
+    for (unsigned i = threadIdx.x; i < c1; i += blockDim.x) gput(wl + b1 + i, st.w[i]);
+    const unsigned nf2 = min(st.nf, (unsigned)kStF);
+    for (unsigned t = threadIdx.x; t < nf2; t += blockDim.x) {
+        const uint2 f = st.fresh[t];
+        const uint2 mt = st.fmeta[t];
+        const int64_t rs = st.frs[t], len = (int64_t)mt.x;
+        const uint32_t fl = kFirst | f.y;
+        if (len <= kShortMax) {
+            Item it;
+            it.v = f.x;
+            it.lf = (uint32_t)len | fl;
+            it.e0 = rs;
+            gput(sl + b0 + c0 + mt.y, it);
+        } else {
+            const uint32_t nseg = (uint32_t)((len + kSeg - 1) / kSeg);
+            const unsigned li = nseg <= kInlineSeg ? (unsigned)kLongMax : atomicAdd(&st.nlong, 1u);
+            if (li < (unsigned)kLongMax) {
+                st.lng[li].rs = rs;
+                st.lng[li].dst = (int64_t)(c1 + mt.y);
+                st.lng[li].w = f.x;
+                st.lng[li].len = (uint32_t)len;
+                st.lng[li].flags = fl;
+            } else {
+                for (uint32_t q = 0; q < nseg; ++q) {
+                    Item si;
+                    si.v = f.x;
+                    si.e0 = rs + (int64_t)q * kSeg;
+                    si.lf = (uint32_t)min((int64_t)kSeg, len - (int64_t)q * kSeg) | (q == 0 ? fl : (fl & kLoSide));
+                    gput(wl + b1 + c1 + mt.y + q, si);
+                }
+            }
+        }
+    }
+    __syncthreads();
+    const unsigned nl = min(st.nlong, (unsigned)kLongMax);
+    for (unsigned r = threadIdx.x >> 5; r < nl; r += blockDim.x >> 5) {  // a warp per long row
+        const Stage::Long L = st.lng[r];
+        const uint32_t nseg = (L.len + kSeg - 1) / kSeg;
+        for (uint32_t q = lane_id(); q < nseg; q += 32) {
+            Item si;
+            si.v = L.w;
+            si.e0 = L.rs + (int64_t)q * kSeg;
+            si.lf = (uint32_t)min((int64_t)kSeg, (int64_t)L.len - (int64_t)q * kSeg) | (q == 0 ? L.flags : (L.flags & kLoSide));
+            gput(wl + b1 + L.dst + q, si);
+        }
+    }
+    // (st.n, st.nd, st.nf are reset at the next round top)
 }
 
 // JP: a mex slot for the long row of w (deg entries): cleared, its
@@ -1407,6 +1517,11 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
                 }
             }
             st.trap = (k & 31u) == 0u ? __ldcg(&a.ctr[cErr]) : 0ull;
+            if (kDirectFlush && !JP && !MH) {  // (the last round's direct flush is done)
+                st.n[0] = st.n[1] = 0;
+                st.nd[0] = st.nd[1] = 0;
+                st.nf = 0;
+            }
             st.rw = round_word(a, (int)((k + 1) % 3), me);
             st.tg_a = tag_a(a.epoch, k + 1u);
             st.tg_b = tag_b(a.epoch, k + 1u);
@@ -1590,8 +1705,12 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
                 }
             }
         }
-        if (!(kEagerFresh && !JP && !MH)) schedule_fresh<JP>(a, prs, t_round);
-        stage_flush(a, prs, t_round, kRelax);
+        if (kDirectFlush && kRelax && !PROF) {
+            fresh_flush_direct(a);
+        } else {
+            if (!(kEagerFresh && !JP && !MH)) schedule_fresh<JP>(a, prs, t_round);
+            stage_flush(a, prs, t_round, kRelax);
+        }
         if (!grid_barrier_rw(a, k, (int)((k + 1) % 3), stage().rd, !kRelax)) return;
         if (PROF && gtid == 0) {
             const unsigned long long t = gtimer();

@@ -35,3 +35,16 @@ tot = np.bincount(r, minlength=R.max() + 1)
 for lo, hi in [(0,1),(1,10),(10,100),(100,1000),(1000,2000),(2000,R.max()+1)]:
     if lo > R.max(): break
     print(lo, hi, 'atomics/round', int(tot[lo:hi].mean()), 'max same-address/round', int(mx[lo:hi].mean()), 'max', int(mx[lo:hi].max()))
+
+# decrements to vertices coloured earlier than the walker, by the target's round
+# (what a residual-row compaction after round K would remove)
+rv = R[src][live]; rw = R[dst][live]
+dead_mask = rw < rv
+print('issued', live.sum(), 'to coloured targets', dead_mask.sum())
+for K in [1, 2, 3, 5, 10, 50]:
+    # compaction at the start of round K removes entries to vertices coloured in rounds < K
+    # from the rows walked in rounds >= K
+    rem = (dead_mask & (rw < K) & (rv >= K)).sum()
+    rows_after = (R >= K)
+    ent_after = deg[rows_after].sum()
+    print(f'compact at round {K}: removes {rem} issued decrements; rows left {rows_after.sum()}, their entries {ent_after}')
