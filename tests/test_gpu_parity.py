@@ -692,3 +692,52 @@ def test_alg2_alg4_scaled(vname):
         g = _csr_tensors(70001, [(i, i + 1) for i in range(70000)])
         C, k, st = gpu_colors(g, 3, gcb.JP_ALG4)
         assert (C == O.color_jp_alg4(g, 3)).all()
+
+
+def _sparse_hubs_graph(n, hubs, hub_deg, leaf_pairs, seed):
+    """Long runs of isolated vertices (more than 32 rows without entries
+    inside one 512-entry warp tile), a few hubs whose rows cross many tiles,
+    and scattered rows of 1-3 entries: the shapes the counting pass's warp
+    tiles walk row chunk by row chunk."""
+    rng = random.Random(seed)
+    pairs = set()
+    for h in hubs:
+        for _ in range(hub_deg):
+            u = rng.randrange(n)
+            if u != h:
+                pairs.add((min(h, u), max(h, u)))
+    for _ in range(leaf_pairs):
+        a, b = rng.randrange(0, n, 97), rng.randrange(n)  # sparse: most rows stay empty
+        if a != b:
+            pairs.add((min(a, b), max(a, b)))
+    return _csr_tensors(n, sorted(pairs))
+
+
+def test_counting_pass_tiles_and_row_runs():
+    """COUNT mode's counting pass (warp tiles over the entries, row chunks of
+    32, rows crossing tile boundaries pre-zeroed, rows without entries left to
+    the init phase) against the oracle, element by element, for max-min and
+    Luby (the same pass with lo pinned), on graphs with long runs of empty
+    rows, hubs spanning many tiles and short rows; several seeds on one
+    handle (the per-graph tile table is reused); a CSR borrowed at a 4-byte
+    offset (not 16-byte aligned: the degree-binned pass) gives the same."""
+    graphs = [_sparse_hubs_graph(60000, [5, 30001, 59999], 6000, 4000, 1),
+              _sparse_hubs_graph(9000, [0, 4500], 2500, 300, 2),
+              G.rmat(14, 4, seed=5)]
+    for g in graphs:
+        with gcb.Graph(g.n, g.row_offsets, g.col_indices) as h:
+            for seed in (1, 7, 123):
+                for vname in ("maxmin", "luby"):
+                    out = torch.empty(g.n, dtype=torch.int32)
+                    _, _, st = h.color(seed, variant_of(vname), out, stats=True, mode=gcb.MODE_COUNT)
+                    assert st.mode_used == gcb.MODE_COUNT
+                    assert (out.numpy().view(np.uint32) == oracle_colors(g, seed, vname)).all(), (g.name, seed, vname)
+    g = graphs[0]
+    ci = torch.empty(g.nnz + 1, dtype=torch.int32, device="cuda")
+    ci[1:] = g.col_indices.to("cuda")
+    ro = g.row_offsets.to("cuda")
+    with gcb.Graph(g.n, ro, ci[1:], flags=gcb.BORROW_DEVICE) as h:
+        out = torch.empty(g.n, dtype=torch.int32, device="cuda")
+        _, _, st = h.color(7, gcb.MAXMIN, out, stats=True, mode=gcb.MODE_COUNT)
+        assert st.mode_used == gcb.MODE_COUNT
+        assert (out.cpu().numpy().view(np.uint32) == O.color_maxmin(g, 7)).all()
