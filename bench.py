@@ -140,6 +140,20 @@ def source_sha(kernel: str) -> str:
         return hashlib.sha256(f.read()).hexdigest()[:16]
 
 
+def atomic_rate_peak():
+    """(G atomics/s, source) of scattered 64-bit atomics with consumed results
+    on a 134 MB array (the s24 count words), measured on this pool's B200 by
+    tools/microbench_atomic_rate.cu (profiles/r02b_microbench_atomic_rate.txt)."""
+    path = os.path.join(ROOT, "profiles", "r02b_microbench_atomic_rate.txt")
+    try:
+        for line in open(path):
+            if "(134 MB)" in line and "G atomics/s" in line:
+                return float(line.split(":")[-1].split()[0]), "measured (" + os.path.relpath(path, ROOT) + ")"
+    except OSError:
+        pass
+    return None
+
+
 def ncu_traffic(workload: str, kernel: str):
     """Per-launch DRAM bytes of `kernel` from a committed ncu --set full capture
     (profiles/ncu_traffic.json, keyed by workload, kernel and the sha of the
@@ -365,6 +379,15 @@ def main():
                              "launches_per_step": 1 if c == 0 else 2,
                              "share_of_step": t_ms / statistics.median(step_ms)}
         classes["k_count_persistent"]["count_decrements"] = A
+        # the same kernel against the measured sustained rate of scattered
+        # 64-bit atomics with consumed results on an array of the count
+        # words' size (tools/microbench_atomic_rate.cu)
+        ar = atomic_rate_peak()
+        if ar:
+            t_ms = statistics.median(kms[0])
+            classes["k_count_persistent"]["atomics"] = {
+                "bound": "l2_atomics", "achieved": A / (t_ms / 1e3) / 1e9, "peak": ar[0], "unit": "G atomics/s",
+                "frac": A / (t_ms / 1e3) / 1e9 / ar[0], "peak_source": ar[1]}
         classes["k_count_persistent"]["bytes_formula"] = "16 n + 56 s + 32 ceil(m/128) + 4 m + 16 A"
         dom = classes["k_count_persistent"]
         roof = dict(dom)
