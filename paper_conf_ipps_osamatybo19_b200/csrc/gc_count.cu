@@ -635,7 +635,10 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
 // a warp each -- while the barrier completes (the items carry round tags the
 // consumers check).  Items staged in shared memory by the rare overflow
 // paths of the walks go first.
-__device__ __forceinline__ void fresh_flush_direct(const CArgs &a) {
+__device__ __forceinline__ void jp_slot_init(const CArgs &a, uint32_t w, int64_t deg);  // (below)
+
+template <bool JP>
+__device__ __forceinline__ void fresh_flush_direct(const CArgs &a, bool relaxed) {
     Stage &st = stage();
     __syncthreads();  // the units are done
     const unsigned nf = min(st.nf, (unsigned)kStF);
@@ -649,6 +652,7 @@ __device__ __forceinline__ void fresh_flush_direct(const CArgs &a) {
             if (!GC_NO_PF_CI && len > 0) asm volatile("prefetch.global.L2 [%0];" ::"l"(a.ci + rs));
         } else {
             pos = atomicAdd(&st.nd[1], (unsigned)((len + kSeg - 1) / kSeg));
+            if (JP && a.jpv == 1) jp_slot_init(a, f.x, len);  // (before the release arrival)
         }
         st.frs[t] = rs;
         st.fmeta[t] = make_uint2((uint32_t)len, pos);
@@ -659,8 +663,10 @@ __device__ __forceinline__ void fresh_flush_direct(const CArgs &a) {
         const unsigned long long t0 = c0 + st.nd[0], t1 = c1 + st.nd[1];
         if (st.colored) atom_add_global(st.ccol, (unsigned long long)st.colored);
         st.colored = 0;
-        // the reservation of both lists is the barrier arrival (relaxed: 7.0)
-        const unsigned long long rv = atom_add_global(st.rw, rw_add(t0, 0) + rw_add(t1, 1) + kRwArr);
+        // the reservation of both lists is the barrier arrival (relaxed for
+        // max-min, 7.0; release for JP, whose mex reads earlier colours)
+        const unsigned long long rv = relaxed ? atom_add_global(st.rw, rw_add(t0, 0) + rw_add(t1, 1) + kRwArr)
+                                              : atom_add_release(st.rw, rw_add(t0, 0) + rw_add(t1, 1) + kRwArr);
         const unsigned long long r0 = rw_field(rv, 0), r1 = rw_field(rv, 1);
         if (r0 + t0 > kMSL || r1 + t1 > kMWL) flag_error(a, 9, 0, 0);  // a round word field overflowed
         st.base[0] = st.nbase[0] + r0;
@@ -706,7 +712,8 @@ __device__ __forceinline__ void fresh_flush_direct(const CArgs &a) {
                     Item si;
                     si.v = f.x;
                     si.e0 = rs + (int64_t)q * kSeg;
-                    si.lf = (uint32_t)min((int64_t)kSeg, len - (int64_t)q * kSeg) | (q == 0 ? fl : (fl & kLoSide));
+                    si.lf = (uint32_t)min((int64_t)kSeg, len - (int64_t)q * kSeg) |
+                            ((q == 0 || (JP && a.jpv == 1)) ? fl : (fl & kLoSide));
                     gput(wl + b1 + c1 + mt.y + q, si);
                 }
             }
@@ -721,7 +728,8 @@ __device__ __forceinline__ void fresh_flush_direct(const CArgs &a) {
             Item si;
             si.v = L.w;
             si.e0 = L.rs + (int64_t)q * kSeg;
-            si.lf = (uint32_t)min((int64_t)kSeg, (int64_t)L.len - (int64_t)q * kSeg) | (q == 0 ? L.flags : (L.flags & kLoSide));
+            si.lf = (uint32_t)min((int64_t)kSeg, (int64_t)L.len - (int64_t)q * kSeg) |
+                    ((q == 0 || (JP && a.jpv == 1)) ? L.flags : (L.flags & kLoSide));
             gput(wl + b1 + L.dst + q, si);
         }
     }
@@ -1517,7 +1525,7 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
                 }
             }
             st.trap = (k & 31u) == 0u ? __ldcg(&a.ctr[cErr]) : 0ull;
-            if (kDirectFlush && !JP && !MH) {  // (the last round's direct flush is done)
+            if (kDirectFlush && !MH && !PROF) {  // (the last round's direct flush is done)
                 st.n[0] = st.n[1] = 0;
                 st.nd[0] = st.nd[1] = 0;
                 st.nf = 0;
@@ -1705,8 +1713,8 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
                 }
             }
         }
-        if (kDirectFlush && kRelax && !PROF) {
-            fresh_flush_direct(a);
+        if (kDirectFlush && !MH && !PROF) {
+            fresh_flush_direct<JP>(a, kRelax);
         } else {
             if (!(kEagerFresh && !JP && !MH)) schedule_fresh<JP>(a, prs, t_round);
             stage_flush(a, prs, t_round, kRelax);
@@ -2096,9 +2104,10 @@ int launch(gc_graph *g, CArgs &a, int *blocks_out) {
         size_t cur = 0;
         cudaDeviceGetLimit(&cur, cudaLimitPersistingL2CacheSize);
         if (cur < (size_t)max_persist) cudaDeviceSetLimit(cudaLimitPersistingL2CacheSize, (size_t)max_persist);
-        const size_t bytes = std::min<size_t>((size_t)a.n * 8, (size_t)max_window);
+        const bool pk = GC_PACKED && !JP && !MH;  // the rounds' count words: 32-bit packed or 64-bit
+        const size_t bytes = std::min<size_t>((size_t)a.n * (pk ? 4 : 8), (size_t)max_window);
         attrs[na].id = cudaLaunchAttributeAccessPolicyWindow;
-        attrs[na].val.accessPolicyWindow.base_ptr = a.cnt;
+        attrs[na].val.accessPolicyWindow.base_ptr = pk ? (void *)a.cnt32 : (void *)a.cnt;
         attrs[na].val.accessPolicyWindow.num_bytes = bytes;
         attrs[na].val.accessPolicyWindow.hitRatio =
             (float)std::min(1.0, (double)max_persist / (double)std::max<size_t>(bytes, 1));
