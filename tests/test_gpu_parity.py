@@ -741,3 +741,45 @@ def test_counting_pass_tiles_and_row_runs():
         _, _, st = h.color(7, gcb.MAXMIN, out, stats=True, mode=gcb.MODE_COUNT)
         assert st.mode_used == gcb.MODE_COUNT
         assert (out.cpu().numpy().view(np.uint32) == O.color_maxmin(g, 7)).all()
+
+
+_OVERFLOW_CHECK = r"""
+import sys
+import numpy as np, torch
+sys.path.insert(0, sys.argv[1])
+import graphgen as G, oracle as O, paper_conf_ipps_osamatybo19_b200 as gcb
+def star(n):
+    return G.csr_from_pairs(n, torch.zeros(n - 1, dtype=torch.int64), torch.arange(1, n, dtype=torch.int64))
+cases = [G.rmat(13, 16, seed=3), G.erdos_renyi(3000, 30000, seed=2), star(20001), G.rmat(16, 16, seed=9)]
+refs = {"maxmin": lambda g: O.color_maxmin(g, 5), "luby": lambda g: O.color_luby(g, 5),
+        "mh3": lambda g: O.color_maxmin(g, 5, 3), "alg2": lambda g: O.color_is_alg2(g, 5),
+        "alg4": lambda g: O.color_jp_alg4(g, 5)}
+codes = {"maxmin": gcb.MAXMIN, "luby": gcb.LUBY_MIS, "mh3": gcb.MULTIHASH(3), "alg2": gcb.IS_ALG2,
+         "alg4": gcb.JP_ALG4}
+for g in cases:
+    with gcb.Graph(g.n, g.row_offsets, g.col_indices) as h:
+        for name, code in codes.items():
+            out = torch.empty(g.n, dtype=torch.int32)
+            _, _, st = h.color(5, code, out, stats=True, mode=gcb.MODE_COUNT)
+            assert st.mode_used == gcb.MODE_COUNT, (g.name, name)
+            assert (out.numpy().view(np.uint32) == refs[name](g)).all(), (g.name, name)
+print("overflow paths ok")
+"""
+
+
+def test_count_overflow_paths(tmp_path):
+    """COUNT rounds from a build whose per-block item staging and fresh list
+    hold 4 / 8 entries (GC_STAGE_ITEMS=4): freed vertices overflow into direct
+    scheduling by the walking warp, staged items spill straight to the global
+    lists, long rows that do not fit leave holes -- paths a normal build takes
+    only in extreme rounds.  Same colourings as the oracle for max-min, Luby,
+    multi-hash, Alg.2 and Alg.4 (a subprocess loads the variant library)."""
+    import subprocess
+    import sys as _sys
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    lib = str(tmp_path / "libgc_stage4.so")
+    gbuild.build(out=lib, defines=["GC_STAGE_ITEMS=4"])
+    env = dict(os.environ, GC_LIB_PATH=lib)
+    r = subprocess.run([_sys.executable, "-c", _OVERFLOW_CHECK, root], env=env, capture_output=True, text=True,
+                       timeout=900)
+    assert r.returncode == 0 and "overflow paths ok" in r.stdout, r.stdout[-2000:] + r.stderr[-4000:]
