@@ -415,7 +415,7 @@ def main():
             names = {0: "k_hash_propose", 1: "k_hash_resolve", 2: "k_hash_table",
                      3: "k_hash_tent + k_hash_commit"}
         if use_dist:
-            names = {0: "k_dc_* round loop (COUNT, host-driven rounds + NCCL all-gathers)"
+            names = {0: "k_dc_persistent (COUNT rounds, device-driven; pairs pushed into the peers' inboxes)"
                      if sp.mode_used == gcb.MODE_COUNT else "sweep round loop",
                      1: "-", 2: "-", 3: "-"}
         if sp.mode_used in (gcb.MODE_EVENT, gcb.MODE_COUNT) or use_dist:
