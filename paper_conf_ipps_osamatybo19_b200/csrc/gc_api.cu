@@ -474,6 +474,7 @@ int gc_create_csr_internal(int64_t n, int64_t nnz, const int64_t *row_offsets,
 
 int gc_create_csr(int64_t n, int64_t nnz, const int64_t *row_offsets, const uint32_t *col_indices,
                   uint32_t flags, gc_graph **out) {
+    NvtxRange nv_("gc_create_csr");
     return gc_create_csr_internal(n, nnz, row_offsets, col_indices, flags, out, 0, n);
 }
 
@@ -504,6 +505,7 @@ void gc_destroy(gc_graph *g) {
 int64_t gc_color_dist(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_stats *stats);
 
 int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_stats *stats) {
+    NvtxRange nv_("gc_color");
     if (!g || !o || o->struct_size < sizeof(gc_options)) {
         set_error("gc_color_ex: NULL handle/options or options.struct_size too small");
         return GC_ERR_INVALID_ARG;

@@ -2235,6 +2235,7 @@ static int ensure_jp_scratch(gc_graph *g) {
 }
 
 static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
+    NvtxRange nv_(jpv ? "COUNT colouring (JP)" : p.H > 1 ? "COUNT colouring (multi-hash)" : "COUNT colouring (max-min)");
     Scratch &s = g->s;
     const int64_t n = g->n;
     const bool jp = jpv != 0;

@@ -100,6 +100,7 @@ int ensure_strict_rows(gc_graph *g) {
 // nnz > 2^31): per batch a segmented sort, the keep flags, an exclusive scan
 // of them (batch-local positions) and the compaction at the running base.
 int dedup_csr(gc_graph *g) {
+    NvtxRange nv_("deduplicate CSR");
     const int64_t n = g->n, m = g->nnz;
     cudaStream_t st = g->stream;
     const int grid = g->sm_count * 8;

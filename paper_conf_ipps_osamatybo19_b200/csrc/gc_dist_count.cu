@@ -911,6 +911,7 @@ bool use_persistent(gc_graph *g) {
 }
 
 int run_dist_persistent(gc_graph *g, const RunParams &p, RunResult *r, int64_t *frontier, int64_t fcap) {
+    NvtxRange nv_("partitioned COUNT rounds (device-driven)");
     Dist &d = *g->dist;
     cudaStream_t st = g->stream;
     const int nlocal = (int)d.parts.size();

@@ -486,6 +486,7 @@ __global__ void __launch_bounds__(kLongThreads) k_hash_table_long(HashArgs a, ui
 }  // namespace
 
 int run_hash_is(gc_graph *g, const RunParams &p, int T, RunResult *r) {
+    NvtxRange nv_("Hash IS colouring");
     Scratch &s = g->s;
     const int64_t n = g->n;
     r->rounds = r->inner = r->launches = 0;

@@ -13,7 +13,19 @@
 #define GC_UNC 0xFFFFFFFFu  // "invalidColor" of Alg.5 L5
 #define GC_MAX_HASHES 16
 
+#include <nvtx3/nvToolsExt.h>  // header-only NVTX 3 (no link dependency; ranges cost ~nothing without a tool)
+
 namespace gc {
+
+// NVTX range for the lifetime of a scope (host side: shows each API call and
+// phase on an Nsight timeline)
+struct NvtxRange {
+    explicit NvtxRange(const char *name) { nvtxRangePushA(name); }
+    ~NvtxRange() { nvtxRangePop(); }
+    NvtxRange(const NvtxRange &) = delete;
+    NvtxRange &operator=(const NvtxRange &) = delete;
+};
+
 
 // ------------------------------------------------------------------ weights
 // R1: p_j(v) = fmix32(v ^ K_j), K_j = fmix32(fold32(seed) +
