@@ -113,6 +113,11 @@ constexpr bool kEagerFresh = GC_EAGER_FRESH != 0;
 #endif
 constexpr bool kDirectFlush = GC_DIRECT_FLUSH != 0;
 
+#ifndef GC_INIT_TWO_PASS
+#define GC_INIT_TWO_PASS 1  // 1: max-min init counts, reserves once per block, then writes round 0's items
+#endif
+constexpr bool kInitTwoPass = GC_INIT_TWO_PASS != 0;
+
 #ifndef GC_PACKED
 #define GC_PACKED 0  // 1: 32-bit (hi << 16 | lo) round counts -- max-min only (no JP / multi-hash branch);
                      // measured 27.9 vs 28.1 ms on R-MAT s24, not worth the restriction
@@ -1375,6 +1380,7 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
     {
         Stage &st = stage();
         if (threadIdx.x < 2) st.n[threadIdx.x] = 0;
+        if (threadIdx.x < 2) st.nd[threadIdx.x] = 0;
         if (threadIdx.x == 0) st.colored = 0;
         if (threadIdx.x == 0) st.vis = 0;
         if (threadIdx.x == 0) st.nf = 0;
@@ -1412,6 +1418,50 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
     // count word and the row offsets of kInitU batches of 32 vertices are
     // loaded together up front (independent loads: the phase is a stream)
     constexpr int kInitU = 4;
+    // max-min (kInit2): a first pass counts the block's round-0 items, ONE
+    // atomic per block reserves them, and the second pass writes each item
+    // straight to its slot -- instead of millions of items spilling from the
+    // block's staging through one round-word atomic per warp append
+    constexpr bool kInit2 = kInitTwoPass && !JP && !MH && !GC_PACKED && kNG == 1;
+    unsigned long long ib0 = 0, ib1 = 0;  // (kInit2) the block's first SL / WL slot of round 0
+    if (kInit2) {
+        // (the same vertices per warp as the second pass below: kInitU batches)
+        for (unsigned long long bb = gwarp * 32 * kInitU; bb < (unsigned long long)n; bb += nwarps * 32 * kInitU)
+        for (int b = 0; b < kInitU; ++b) {
+            const unsigned long long vv = bb + 32ull * b + lane;
+            bool zero = false;
+            int64_t len = 0;
+            if (vv < (unsigned long long)n) {
+                const int64_t rs = __ldg(a.ro + vv), re = __ldg(a.ro + vv + 1);
+                len = re - rs;
+                if (len > 0) {
+                    const unsigned long long c = __ldcs(a.cnt + vv);
+                    zero = (uint32_t)(c >> 32) == 0u || (uint32_t)c == 0u;
+                }
+            }
+            const unsigned nsl = __popc(__ballot_sync(kFull, zero && len <= kShortMax));
+            const unsigned nwl = __reduce_add_sync(kFull, (zero && len > kShortMax) ? (unsigned)((len + kSeg - 1) / kSeg) : 0u);
+            if (lane == 0) {
+                if (nsl) atomicAdd(&stage().nd[0], nsl);
+                if (nwl) atomicAdd(&stage().nd[1], nwl);
+            }
+        }
+        __syncthreads();
+        Stage &st = stage();
+        if (threadIdx.x == 0) {
+            const unsigned long long t0i = st.nd[0], t1i = st.nd[1];
+            const unsigned long long rv = (t0i || t1i) ? atom_add_global(st.rw, rw_add(t0i, 0) + rw_add(t1i, 1)) : 0ull;
+            const unsigned long long r0 = rw_field(rv, 0), r1 = rw_field(rv, 1);
+            if (r0 + t0i > kMSL || r1 + t1i > kMWL) flag_error(a, 9, 0, 0);
+            if (r0 + t0i > a.sl_cap || r1 + t1i > a.wl_cap) flag_error(a, 2, 0, 0);
+            st.base[0] = r0;
+            st.base[1] = r1;
+            st.nd[0] = st.nd[1] = 0;  // now the position counters
+        }
+        __syncthreads();
+        ib0 = st.base[0];
+        ib1 = st.base[1];
+    }
     for (unsigned long long base0 = gwarp * 32 * kInitU; base0 < (unsigned long long)n;
          base0 += nwarps * 32 * kInitU) {
       unsigned long long cpre[kInitU];
@@ -1478,8 +1528,50 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
         }
         if (lane == 0 && word) atomicAdd(&stage().colored, (unsigned)__popc(word));
         // walked in round 0 (the free side's flag: its neighbours, if any, are dead)
-        schedule_rows<JP>(a, zero && re > rs, v, rs, re - rs, (!JP && !MH && lo == 0u) ? kLoSide : 0u);
+        if (kInit2) {
+            const uint32_t fl = lo == 0u ? kLoSide : 0u;
+            const int64_t len = re - rs;
+            const bool sl = zero && len > 0 && len <= kShortMax;
+            const unsigned msl = __ballot_sync(kFull, sl);
+            if (msl) {
+                unsigned p0 = 0;
+                if (lane == (unsigned)(__ffs(msl) - 1)) p0 = atomicAdd(&stage().nd[0], (unsigned)__popc(msl));
+                p0 = __shfl_sync(kFull, p0, __ffs(msl) - 1);
+                if (sl) {
+                    Item it;
+                    it.v = v;
+                    it.lf = (uint32_t)len | fl;
+                    it.e0 = rs;
+                    gput(a.SL + ib0 + p0 + __popc(msl & ((1u << lane) - 1u)), it);
+                }
+            }
+            const bool lg = zero && len > kShortMax;
+            const uint32_t nseg = lg ? (uint32_t)((len + kSeg - 1) / kSeg) : 0u;
+            const unsigned pw = lg ? atomicAdd(&stage().nd[1], nseg) : 0u;
+            unsigned lm = __ballot_sync(kFull, lg);
+            while (lm) {  // the warp writes each long row's segments
+                const int src = __ffs(lm) - 1;
+                lm &= lm - 1;
+                const uint32_t ww = __shfl_sync(kFull, v, src);
+                const int64_t r0 = __shfl_sync(kFull, rs, src), ln = __shfl_sync(kFull, len, src);
+                const uint32_t fs = __shfl_sync(kFull, fl, src), ns = __shfl_sync(kFull, nseg, src);
+                const unsigned ps = __shfl_sync(kFull, pw, src);
+                for (uint32_t q = lane; q < ns; q += 32) {
+                    Item si;
+                    si.v = ww;
+                    si.e0 = r0 + (int64_t)q * kSeg;
+                    si.lf = (uint32_t)min((int64_t)kSeg, ln - (int64_t)q * kSeg) | fs;
+                    gput(a.WL + ib1 + ps + q, si);
+                }
+            }
+        } else {
+            schedule_rows<JP>(a, zero && re > rs, v, rs, re - rs, (!JP && !MH && lo == 0u) ? kLoSide : 0u);
+        }
       }
+    }
+    if (kInit2) {  // (the items are written; the arrival below reserves none)
+        __syncthreads();
+        if (threadIdx.x == 0) stage().nd[0] = stage().nd[1] = 0;
     }
     stage_flush(a);
     if (!grid_barrier_rw(a, 0, 0, stage().rd)) return;
