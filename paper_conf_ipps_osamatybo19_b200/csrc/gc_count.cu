@@ -234,6 +234,7 @@ struct CArgs {
     uint32_t mkeys[GC_MAX_HASHES]; // MH: their keys K_j
     const uint32_t *dg;            // LDF: vertex degrees; nullptr = weights only
     uint32_t epoch;                // colourings run on this handle (item round tags)
+    int jrel;                      // JP Luby / Alg.2 rounds relaxed (jp_colour_of, jp_segment_done)
 };
 
 // Round tags of the items walked in round r (merged hand-off): items are
@@ -749,11 +750,30 @@ __device__ __forceinline__ void jp_slot_init(const CArgs &a, uint32_t w, int64_t
         flag_error(a, 6, 0, w);
         return;
     }
-    uint4 *p = reinterpret_cast<uint4 *>(a.jslot + s * kSlotWords);
+    if (!a.jrel) {  // (relaxed rounds: the host zeroes every slot before the colouring)
+        uint4 *p = reinterpret_cast<uint4 *>(a.jslot + s * kSlotWords);
 #pragma unroll
-    for (int i = 0; i < kSlotWords / 4; ++i) p[i] = make_uint4(0u, 0u, 0u, 0u);
-    a.jslot[s * kSlotWords + 32] = (uint32_t)deg;
+        for (int i = 0; i < kSlotWords / 4; ++i) p[i] = make_uint4(0u, 0u, 0u, 0u);
+        a.jslot[s * kSlotWords + 32] = (uint32_t)deg;
+    }
     a.Zlo[w] = (uint32_t)s;
+}
+
+// JP, relaxed rounds: a value written once in an earlier round by another
+// block (a predecessor's colour, a row's slot index) is read until it is no
+// longer the initial one -- a single-writer word that changes once, so the
+// value read then is the value written, whatever the ordering
+__device__ __forceinline__ uint32_t jp_read_once(const CArgs &a, const uint32_t *p, uint32_t init, uint32_t k,
+                                                 uint32_t v) {
+    uint32_t x = __ldcg(p);
+    for (unsigned spins = 0; x == init; ++spins) {
+        if (spins > (1u << 22)) {  // (~ms: the writer's round is long over -- cannot happen)
+            flag_error(a, 5, k, v);
+            break;
+        }
+        x = __ldcg(p);
+    }
+    return x;
 }
 
 // Whole warp converged: schedule the rows of the lanes with `pred` (vertex w,
@@ -901,9 +921,13 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint64_t pv, in
     if (JP && want_mex) {
 #pragma unroll
         for (int q = 0; q < Q; ++q) {
+            if (w[q] != kNone && !hi[q] && cv[q] == GC_UNC) {
+                // a predecessor's colour not seen yet (relaxed rounds) or an uncoloured predecessor (error)
+                if (a.jrel) cv[q] = jp_read_once(a, a.C + w[q], GC_UNC, k, v);
+                else flag_error(a, 5, k, v);
+            }
             const uint32_t c = cv[q];
             if (w[q] != kNone && !hi[q]) {
-                if (c == GC_UNC) flag_error(a, 5, k, v);  // a predecessor is uncoloured
                 if (WIDE) {
                     if (c < 1024u) atomicOr(sbits + (c >> 5), 1u << (c & 31u));
                 } else if (c < 64u) {
@@ -1262,10 +1286,10 @@ __device__ __forceinline__ void schedule_fresh(const CArgs &a, int64_t *prs = nu
 __device__ __noinline__ uint32_t jp_mex_rescan(const CArgs &a, uint32_t v, uint64_t pv, uint32_t *sb);
 
 __device__ __forceinline__ void jp_segment_done(const CArgs &a, uint32_t v, uint32_t len, uint64_t pv,
-                                                uint32_t *sb, uint32_t k) {
+                                                uint32_t *sb, uint32_t k, int64_t deg) {
     const unsigned lane = lane_id();
     __syncwarp();
-    const uint32_t slot = __ldcg(a.Zlo + v);
+    const uint32_t slot = a.jrel ? jp_read_once(a, a.Zlo + v, kNever, k, v) : __ldcg(a.Zlo + v);
     uint32_t *S = a.jslot + (size_t)slot * kSlotWords;
     const uint32_t word = sb[lane];
     if (word) atomicOr(S + lane, word);
@@ -1274,10 +1298,17 @@ __device__ __forceinline__ void jp_segment_done(const CArgs &a, uint32_t v, uint
     uint32_t last = 0;
     if (lane == 0) {
         uint32_t old;
-        asm volatile("atom.acq_rel.gpu.global.add.u32 %0, [%1], %2;"
-                     : "=r"(old) : "l"(S + 32), "r"(0u - len) : "memory");
-        last = old == len ? 1u : 0u;
-        if (old < len) flag_error(a, 7, k, v);
+        if (a.jrel) {  // count up from the host's zero: the segment that completes the row is last
+            asm volatile("atom.acq_rel.gpu.global.add.u32 %0, [%1], %2;"
+                         : "=r"(old) : "l"(S + 32), "r"(len) : "memory");
+            last = (int64_t)old + len == deg ? 1u : 0u;
+            if ((int64_t)old + len > deg) flag_error(a, 7, k, v);
+        } else {
+            asm volatile("atom.acq_rel.gpu.global.add.u32 %0, [%1], %2;"
+                         : "=r"(old) : "l"(S + 32), "r"(0u - len) : "memory");
+            last = old == len ? 1u : 0u;
+            if (old < len) flag_error(a, 7, k, v);
+        }
     }
     last = __shfl_sync(kFull, last, 0);
     if (!last) return;
@@ -1309,7 +1340,7 @@ __device__ __noinline__ uint32_t jp_mex_rescan(const CArgs &a, uint32_t v, uint6
         for (int64_t e = rs + lane; e < re; e += 32) {
             const uint32_t u = a.ci[e];
             if (prio_key(a, u) > pv) {
-                const uint32_t c = __ldcg(a.C + u) - b;
+                const uint32_t c = (a.jrel ? jp_read_once(a, a.C + u, GC_UNC, 0u, v) : __ldcg(a.C + u)) - b;
                 if (c < kMexWin) atomicOr(sb + (c >> 5), 1u << (c & 31u));
             }
         }
@@ -1374,6 +1405,9 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
     // in the rounds are provisional (max unless the item's side is lo) and
     // the lo-freed-second stamps are applied after the rounds (colour_final)
     constexpr bool kRelax = kRelaxedArrive && !JP && !MH;
+    // relaxed rounds at run time: max-min always, JP for Luby and Alg.2 (a.jrel:
+    // the values a later round reads are read until written, jp_read_once)
+    const bool relax = kRelax || (JP && a.jrel);
     uint32_t nvis = 0;
     unsigned long long nvis_tot = 0, t_rounds = 0;
     unsigned long long t0 = PROF ? gtimer() : 0ull;
@@ -1512,7 +1546,7 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
                 a.Zlo[v] = code;  // round 0's decision (not kNever: never rescheduled)
                 a.C[v] = zero ? 2u * (code >> 1) + ((code & 1u) ? 0u : 1u) : GC_UNC;
             } else {
-                if (!JP) a.Zlo[v] = kNever;
+                if (!JP || a.jrel) a.Zlo[v] = kNever;
                 a.C[v] = zero ? (lo == 0u ? 1u : 0u) : GC_UNC;
             }
             if (zero) {
@@ -1667,10 +1701,12 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
                 } else if (JP && (it.lf & kFirst)) {  // a segment of a row being coloured
                     uint32_t *sb = stage().wbits[threadIdx.x >> 5];
                     sb[lane] = 0u;
+                    // (relaxed rounds: the row's length for the count-up completion, loaded now)
+                    const int64_t dgv = a.jrel ? __ldg(a.ro + it.v + 1) - __ldg(a.ro + it.v) : 0;
                     __syncwarp();
                     walk<kSeg / 32, true, true>(a, it.v, pv, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k,
                                                 nvis, nullptr, sb, true);
-                    jp_segment_done(a, it.v, it.lf & kLenMask, pv, sb, k);
+                    jp_segment_done(a, it.v, it.lf & kLenMask, pv, sb, k, dgv);
                 } else {
                     const bool cl = !JP && (it.lf & kFirst) && lane == 0;
                     const uint32_t z = (cl && !kRelax) ? __ldcg(a.Zlo + it.v) : kNever;
@@ -1806,12 +1842,12 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
             }
         }
         if (kDirectFlush && !MH && !PROF) {
-            fresh_flush_direct<JP>(a, kRelax);
+            fresh_flush_direct<JP>(a, relax);
         } else {
             if (!(kEagerFresh && !JP && !MH)) schedule_fresh<JP>(a, prs, t_round);
-            stage_flush(a, prs, t_round, kRelax);
+            stage_flush(a, prs, t_round, relax);
         }
-        if (!grid_barrier_rw(a, k, (int)((k + 1) % 3), stage().rd, !kRelax)) return;
+        if (!grid_barrier_rw(a, k, (int)((k + 1) % 3), stage().rd, !relax)) return;
         if (PROF && gtid == 0) {
             const unsigned long long t = gtimer();
             if ((int64_t)k < a.nk_cap) a.rstat[16 * k + 4] = (int64_t)(t - t0);
@@ -1820,7 +1856,7 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
         }
     }
     (void)wpb;
-    if (kRelax) {
+    if (relax) {
         // one release / acquire barrier (every block's stamps and colours are
         // visible), then each colour of round k >= 1 that was written as the
         // max 2k becomes the min 2k+1 if v's lo side was freed second by
@@ -1844,7 +1880,7 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
             const uint32_t c = __ldcg(a.C + v);
             if (c == GC_UNC) continue;
             ++ncol;
-            if ((c & 1u) == 0u && __ldcg(a.Zlo + v) <= (c >> 1)) a.C[v] = c | 1u;
+            if (!JP && (c & 1u) == 0u && __ldcg(a.Zlo + v) <= (c >> 1)) a.C[v] = c | 1u;
         }
         const unsigned s = __reduce_add_sync(kFull, ncol);
         if (lane == 0 && s) atomicAdd(&a.ctr[cCol], (unsigned long long)s);
@@ -1864,7 +1900,7 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
         a.ctr[cIters] = k;
         // the colourings of round k-1 (init's for k == 0) not yet subtracted
         rem -= (int64_t)__ldcg(&a.ctr[cK + 16 * (k == 0 ? 0 : (int)((k + 2) % 3))]);
-        if (!kRelax) a.ctr[cCol] = (unsigned long long)(n - rem);
+        if (!relax) a.ctr[cCol] = (unsigned long long)(n - rem);
         if (PROF) a.ctr[cPhaseNs + 1] = t_rounds;
     }
     {
@@ -2444,6 +2480,11 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
         ++s.count_epoch;
     }
     a.epoch = s.count_epoch;
+    // JP rounds relaxed for Luby and Alg.2 (Alg.4's per-round colour sets stay
+    // behind release / acquire barriers); Luby's mex slots zeroed up front
+    a.jrel = (jp && jpv != 3 && kRelaxedArrive && !std::getenv("GC_JP_NO_RELAX")) ? 1 : 0;
+    if (a.jrel && jpv == 1 && s.jslot)
+        GC_CUDA_TRY(cudaMemsetAsync(s.jslot, 0, ((size_t)s.jslot_cap + 1) * kSlotWords * 4, st));
     a.M = s.cM;
     a.jpv = jpv;
     a.cr = nullptr;
