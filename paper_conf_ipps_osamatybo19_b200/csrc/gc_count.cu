@@ -1032,7 +1032,7 @@ __device__ __forceinline__ void walk(const CArgs &a, uint32_t v, uint64_t pv, in
 // schedules w (exactly one per vertex).
 template <int Q>
 __device__ __forceinline__ void walk_mh(const CArgs &a, uint32_t v, int64_t e, int64_t end, int stride,
-                                        uint32_t k, uint32_t &nvis) {
+                                        uint32_t k, uint32_t &nvis, uint32_t zdec = kNever) {
     uint32_t w[Q];
 #pragma unroll
     for (int q = 0; q < Q; ++q) {
@@ -1040,6 +1040,17 @@ __device__ __forceinline__ void walk_mh(const CArgs &a, uint32_t v, int64_t e, i
         w[q] = (v != kNone && eq < end) ? __ldcs(a.ci + eq) : kNone;
     }
     const int H = a.H;
+    if (kSkipDead && v != kNone && zdec != kNever) {
+        // dead side (walk()): v's decision code names the weight function j
+        // and the side of v that was free under it -- every neighbour on that
+        // side is coloured, so none of its H counts needs a decrement
+        const uint32_t js = (zdec >> 1) & 15u;
+        const bool hifree = (zdec & 1u) != 0u;
+        const uint32_t pvs = weight_mix(v ^ a.mkeys[js]);
+#pragma unroll
+        for (int q = 0; q < Q; ++q)
+            if (w[q] != kNone && (pvs > weight_mix(w[q] ^ a.mkeys[js])) != hifree) w[q] = kNone;
+    }
     if (GC_SKIP_COLOURED) {
         uint32_t mb[Q];
 #pragma unroll
@@ -1716,7 +1727,8 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
                         tp[2] = clock64();
                     }
                     if (MH)
-                        walk_mh<kSeg / 32>(a, it.v, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k, nvis);
+                        walk_mh<kSeg / 32>(a, it.v, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k, nvis,
+                                           it.v != kNone ? __ldcg(a.Zlo + it.v) : kNever);
                     else
                         walk<kSeg / 32, JP>(a, it.v, pv, it.e0 + lane, it.e0 + (it.lf & kLenMask), 32, k, nvis,
                                             nullptr, nullptr, false, false, (GC_PROF_UNIT && prs) ? tp : nullptr,
@@ -1760,8 +1772,9 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
                     if (cl && !kRelax) z = __ldcg(a.Zlo + v);
                 }
                 unsigned long long mask = 0ull;
+                const uint32_t zm = (MH && v != kNone) ? __ldcg(a.Zlo + v) : kNever;  // (MH: v's decision)
                 for (uint32_t j = 0; __any_sync(kFull, j < len); j += 4) {
-                    if (MH) walk_mh<4>(a, j < len ? v : kNone, e0 + j, e0 + len, 1, k, nvis);
+                    if (MH) walk_mh<4>(a, j < len ? v : kNone, e0 + j, e0 + len, 1, k, nvis, zm);
                     else walk<4, JP>(a, j < len ? v : kNone, pv, e0 + j, e0 + len, 1, k, nvis, &mask, nullptr, want,
                                      JP && a.jpv == 3, nullptr, JP ? -1 : ((lf & kLoSide) ? 1 : 0));
                 }
@@ -1794,7 +1807,8 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
                     if (cl && !kRelax) z = __ldcg(a.Zlo + v);
                 }
                 unsigned long long mask = 0ull;
-                if (MH) walk_mh<4>(a, v, e0 + (lane & 7u), e0 + len, 8, k, nvis);
+                const uint32_t zm = (MH && v != kNone) ? __ldcg(a.Zlo + v) : kNever;  // (MH: v's decision)
+                if (MH) walk_mh<4>(a, v, e0 + (lane & 7u), e0 + len, 8, k, nvis, zm);
                 else walk<4, JP>(a, v, pv, e0 + (lane & 7u), e0 + len, 8, k, nvis, &mask, nullptr, want,
                                  JP && a.jpv == 3, nullptr, JP ? -1 : ((lf & kLoSide) ? 1 : 0));
                 if (cl) colour_fin<MH>(a, v, lf, k, z);
