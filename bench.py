@@ -295,7 +295,9 @@ def main():
         from paper_conf_ipps_osamatybo19_b200 import dist as gdist
         g, handle, n, nnz_global = gdist.build_partitioned_rmat(scale, 16, 1, rank, world, dev)
     else:
-        g = G.rmat(scale, 16, seed=1, device=dev)
+        # (scale >= 26: built row range by row range -- torch.unique / CUB take
+        # < 2^32 entries at once; the same CSR)
+        g = G.rmat(scale, 16, seed=1, device=dev, pieces=1 if scale < 26 else 1 << (scale - 25))
         n, nnz_global = g.n, g.nnz
         handle = gcb.Graph(g.n, g.row_offsets, g.col_indices, flags=gcb.BORROW_DEVICE)
     torch.cuda.synchronize()
