@@ -2139,10 +2139,30 @@ __global__ void __launch_bounds__(kWT) k_count_warp(const int64_t *__restrict__ 
         for (int q = 0; q < kWQ; ++q) mx[q] = weight_mix(u[q] ^ key);
         int cur = 0;  // this lane's entries < cur are counted
         for (int64_t rb = ra; rb <= rz; rb += 32) {
-            const int nr = (int)min((int64_t)32, rz - rb + 1);
+            int nr = (int)min((int64_t)32, rz - rb + 1);
             offs[lane] = lane <= nr ? (long long)__ldg(ro + rb + lane) : 0ll;
             if (lane == 0) offs[32] = nr == 32 ? (long long)__ldg(ro + rb + 32) : 0ll;
             __syncwarp();
+            if (nr == 32 && offs[0] == offs[32] && rb + 32 <= rz) {
+                // 32 rows without entries and more to come (a run of isolated
+                // vertices): jump to the last empty row before the next row with
+                // entries (binary search in the offsets; empty rows are the init
+                // phase's), so a long run costs log n, not n / 32, steps
+                const long long e = offs[0];
+                int64_t lo = rb + 32, hi = rz + 1;  // ro[lo] == e; the first r with ro[r] > e is in (lo, hi]
+                if (__ldg(ro + hi) == e) {
+                    rb = rz + 1 - 32;  // (no entries up to rz + 1: nothing left in this tile)
+                } else {
+                    while (hi - lo > 1) {
+                        const int64_t mid = lo + ((hi - lo) >> 1);
+                        if (__ldg(ro + mid) == e) lo = mid;
+                        else hi = mid;
+                    }
+                    rb = lo - 32;  // ro[lo] == e < ro[lo + 1]: row lo is the next with entries; += 32 lands on it
+                }
+                __syncwarp();
+                continue;
+            }
             const int64_t lim = min((int64_t)offs[nr], e1);  // entries of these rows within the tile
             // this lane's entries [cur, qlim) of these rows, one row per step:
             // the row's hi count = popcount of the entries whose priority beats

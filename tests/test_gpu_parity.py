@@ -783,3 +783,27 @@ def test_count_overflow_paths(tmp_path):
     r = subprocess.run([_sys.executable, "-c", _OVERFLOW_CHECK, root], env=env, capture_output=True, text=True,
                        timeout=900)
     assert r.returncode == 0 and "overflow paths ok" in r.stdout, r.stdout[-2000:] + r.stderr[-4000:]
+
+
+def test_counting_pass_long_isolated_runs():
+    """Millions of isolated vertices between a few edges (one warp tile spans
+    them all): the counting pass jumps over runs of empty rows by binary
+    search instead of walking them 32 at a time; same colourings as the
+    oracle, and an edgeless graph of 2^22 vertices colours fast."""
+    import time
+    n = 3_000_000
+    pairs = [(0, 1), (1, 2), (2, 3), (0, 3), (5, n - 7), (n - 3, n - 2), (n - 2, n - 1), (17, n // 2), (n // 2, n // 2 + 1)]
+    g = _csr_tensors(n, pairs)
+    for vname in ("maxmin", "luby"):
+        C, _, st = gpu_colors(g, 3, variant_of(vname), mode=gcb.MODE_COUNT)
+        assert st.mode_used == gcb.MODE_COUNT
+        assert (C == oracle_colors(g, 3, vname)).all(), vname
+    e = G.csr_from_lists(1 << 22, [])
+    with gcb.Graph(e.n, e.row_offsets, e.col_indices) as h:
+        out = torch.empty(e.n, dtype=torch.int32)
+        h.color(1, gcb.MAXMIN, out, mode=gcb.MODE_COUNT)
+        t0 = time.perf_counter()
+        _, k, st = h.color(2, gcb.MAXMIN, out, stats=True, mode=gcb.MODE_COUNT)
+        dt = time.perf_counter() - t0
+    assert k == 1 and st.rounds == 1 and (out.numpy() == 1).all()
+    assert dt < 0.5, dt
