@@ -140,6 +140,26 @@ __global__ void k_mark(const uint32_t *__restrict__ C, int64_t n, uint32_t *bitm
     }
 }
 
+// the same with the block's share of the used-colour set in shared memory
+// (every SM otherwise keeps re-issuing atomics on the few hundred global
+// words: its L1 copy of a word never shows other SMs' bits); one OR per
+// non-zero word and block at the end
+constexpr int64_t kMarkSmemWords = 12288;  // 48 KB: colours < 393,216
+__global__ void k_mark_sm(const uint32_t *__restrict__ C, int64_t n, uint32_t *bitmap, int64_t words) {
+    extern __shared__ uint32_t sb[];
+    for (int64_t i = threadIdx.x; i < words; i += blockDim.x) sb[i] = 0u;
+    __syncthreads();
+    for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n;
+         i += (int64_t)gridDim.x * blockDim.x) {
+        const uint32_t c = C[i];
+        const uint32_t bit = 1u << (c & 31);
+        if (!(sb[c >> 5] & bit)) atomicOr(&sb[c >> 5], bit);
+    }
+    __syncthreads();
+    for (int64_t i = threadIdx.x; i < words; i += blockDim.x)
+        if (sb[i]) atomicOr(&bitmap[i], sb[i]);
+}
+
 __global__ void k_popc(const uint32_t *__restrict__ bitmap, int64_t words, unsigned long long *cnt) {
     unsigned long long s = 0;
     for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < words;
@@ -300,7 +320,13 @@ int64_t count_colors_device(gc_graph *g, const uint32_t *C, int64_t n, bool comp
     }
     uint32_t *rank = s.bitmap + words;
     GC_CUDA_TRY(cudaMemsetAsync(s.bitmap, 0, (size_t)words * 4, st));
-    k_mark<<<grid, 256, 0, st>>>(C, n, s.bitmap);
+    if (words <= kMarkSmemWords) {
+        if (words * 4 > 48 * 1024)
+            GC_CUDA_TRY(cudaFuncSetAttribute(k_mark_sm, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)(words * 4)));
+        k_mark_sm<<<std::min<int>(grid, g->sm_count * 4), 512, (size_t)words * 4, st>>>(C, n, s.bitmap, words);
+    } else {
+        k_mark<<<grid, 256, 0, st>>>(C, n, s.bitmap);
+    }
     k_popc<<<grid_for(words, g->sm_count), 256, 0, st>>>(s.bitmap, words, tmp + 1);
     *launches += 3;
     if (compact) {
