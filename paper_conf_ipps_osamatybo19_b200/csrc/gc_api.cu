@@ -295,18 +295,23 @@ int ensure_scratch(gc_graph *g, bool need_event, bool need_luby) {
 
 // Distinct colours of C[0..n); optionally renumber in place (R12).
 int64_t count_colors_device(gc_graph *g, const uint32_t *C, int64_t n, bool compact,
-                            uint32_t *C_inout, int64_t *launches) {
+                            uint32_t *C_inout, int64_t *launches, int64_t max_hint) {
     if (n == 0) return 0;
     Scratch &s = g->s;
     cudaStream_t st = g->stream;
     unsigned long long *tmp = s.ctr + 48;
     GC_CUDA_TRY(cudaMemsetAsync(tmp, 0, 2 * sizeof(unsigned long long), st));
     const int grid = grid_for(n, g->sm_count);
-    k_max_u32<<<grid, 256, 0, st>>>(C, n, tmp);
-    GC_CUDA_TRY(cudaMemcpyAsync(s.host_pinned, tmp, sizeof(unsigned long long),
-                                cudaMemcpyDeviceToHost, st));
-    GC_CUDA_TRY(cudaStreamSynchronize(st));
-    const uint64_t maxc = *reinterpret_cast<unsigned long long *>(s.host_pinned);
+    uint64_t maxc;
+    if (max_hint >= 0) {  // (the colouring kernel computed it: no pass, no host round trip)
+        maxc = (uint64_t)max_hint;
+    } else {
+        k_max_u32<<<grid, 256, 0, st>>>(C, n, tmp);
+        GC_CUDA_TRY(cudaMemcpyAsync(s.host_pinned, tmp, sizeof(unsigned long long),
+                                    cudaMemcpyDeviceToHost, st));
+        GC_CUDA_TRY(cudaStreamSynchronize(st));
+        maxc = *reinterpret_cast<unsigned long long *>(s.host_pinned);
+    }
     if (maxc == GC_UNC) {
         set_error("internal: uncoloured vertex in the result");
         return GC_ERR_CUDA;
@@ -693,7 +698,7 @@ int64_t gc_color_ex(gc_graph *g, const gc_options *o, int32_t *colors_out, gc_st
     if (rc) return rc;
     int64_t launches = res.launches;
     int64_t ncol = count_colors_device(g, g->s.C, g->n, (o->flags & GC_COMPACT) != 0, g->s.C,
-                                       &launches);
+                                       &launches, res.max_color);
     if (ncol < 0) return ncol;
     if (g->n > 0) {
         GC_CUDA_TRY(cudaMemcpyAsync(colors_out, g->s.C, sizeof(int32_t) * (size_t)g->n,

@@ -190,6 +190,7 @@ enum : int {
     cCol = 144,     // vertices coloured (written at the end, host check)
     cBar = 160,     // (unused: arrivals live in the round words)
     cFin = 168,     // relaxed rounds: the final release / acquire barrier
+    cMaxC = 171,    // relaxed rounds: 1 + the largest colour (0: none)
     cAbort = 176,
     cErr = 192,     // [192..194] first trap: kind, round, vertex
     cRounds = 208,  // result: rounds R
@@ -1889,15 +1890,19 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
             }
         }
         __syncthreads();
-        uint32_t ncol = 0;
+        uint32_t ncol = 0, cmax = 0;
         for (unsigned long long v = gtid; v < (unsigned long long)n; v += nthreads) {
-            const uint32_t c = __ldcg(a.C + v);
+            uint32_t c = __ldcg(a.C + v);
             if (c == GC_UNC) continue;
             ++ncol;
-            if (!JP && (c & 1u) == 0u && __ldcg(a.Zlo + v) <= (c >> 1)) a.C[v] = c | 1u;
+            if (!JP && (c & 1u) == 0u && __ldcg(a.Zlo + v) <= (c >> 1)) a.C[v] = (c |= 1u);
+            cmax = max(cmax, c);
         }
         const unsigned s = __reduce_add_sync(kFull, ncol);
         if (lane == 0 && s) atomicAdd(&a.ctr[cCol], (unsigned long long)s);
+        // the largest colour (the distinct-colour count sizes its set with it)
+        const unsigned mx = __reduce_max_sync(kFull, cmax);
+        if (lane == 0 && s) atomicMax(&a.ctr[cMaxC], (unsigned long long)mx + 1ull);
     }
     if (JP && a.jpv == 3) {
         // colours were round indices: C[v] <- colour of its round (the last
@@ -2403,6 +2408,7 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
     const bool jp = jpv != 0;
     const bool mh = !jp && p.H > 1;
     r->rounds = r->inner = r->launches = 0;
+    r->max_color = -1;  // (set only by a run that completes)
     if (n == 0) return GC_OK;
     if (n >= (1ll << 29)) {  // a round's SL items could pass the round word's 29-bit field
         set_error("COUNT mode: n >= 2^29 exceeds the round word's item field");
@@ -2568,6 +2574,7 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
         return GC_ERR_NOT_SYMMETRIC;
     }
     r->rounds = (int64_t)h[cRounds];
+    r->max_color = h[cMaxC] ? (int64_t)h[cMaxC] - 1 : -1;  // (relaxed rounds' final pass)
     r->inner = r->rounds;
     if (p.prof) {
         // class 0: the persistent kernel; 1: counting kernels (both timed on

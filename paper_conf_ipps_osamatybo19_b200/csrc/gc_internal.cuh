@@ -196,6 +196,7 @@ struct RunResult {
     int64_t rounds = 0;
     int64_t inner = 0;
     int64_t launches = 0;
+    int64_t max_color = -1;  // the largest colour, when the run computed it (else -1)
 };
 
 // One sweep round over a vertex range [v0, v0 + n_loc) (single GPU: v0 = 0).
@@ -233,7 +234,7 @@ int run_count_jp(gc_graph *g, const RunParams &p, RunResult *r, int jpv);  // 1 
 int run_luby(gc_graph *g, const RunParams &p, RunResult *r);
 int run_hash_is(gc_graph *g, const RunParams &p, int T, RunResult *r);  // gc_hash.cu (Alg.6)
 int64_t count_colors_device(gc_graph *g, const uint32_t *C, int64_t n, bool compact,
-                            uint32_t *C_inout, int64_t *launches);
+                            uint32_t *C_inout, int64_t *launches, int64_t max_hint = -1);
 int launch_priorities(uint64_t seed, int j, int64_t v_begin, int64_t count, uint32_t *out,
                       cudaStream_t st);
 
