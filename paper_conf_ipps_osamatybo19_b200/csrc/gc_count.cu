@@ -1471,26 +1471,30 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
     constexpr bool kInit2 = kInitTwoPass && !JP && !MH && !GC_PACKED && kNG == 1;
     unsigned long long ib0 = 0, ib1 = 0;  // (kInit2) the block's first SL / WL slot of round 0
     if (kInit2) {
-        // (the same vertices per warp as the second pass below: kInitU batches)
-        for (unsigned long long bb = gwarp * 32 * kInitU; bb < (unsigned long long)n; bb += nwarps * 32 * kInitU)
-        for (int b = 0; b < kInitU; ++b) {
+        // (the same vertices per warp as the second pass below: kInitU batches,
+        // their count words and offsets loaded together up front)
+        for (unsigned long long bb = gwarp * 32 * kInitU; bb < (unsigned long long)n; bb += nwarps * 32 * kInitU) {
+          unsigned long long cq[kInitU];
+          int64_t lq[kInitU];
+#pragma unroll
+          for (int b = 0; b < kInitU; ++b) {
             const unsigned long long vv = bb + 32ull * b + lane;
-            bool zero = false;
-            int64_t len = 0;
-            if (vv < (unsigned long long)n) {
-                const int64_t rs = __ldg(a.ro + vv), re = __ldg(a.ro + vv + 1);
-                len = re - rs;
-                if (len > 0) {
-                    const unsigned long long c = __ldcs(a.cnt + vv);
-                    zero = (uint32_t)(c >> 32) == 0u || (uint32_t)c == 0u;
-                }
-            }
+            const bool ok = vv < (unsigned long long)n;
+            cq[b] = ok ? __ldcg(a.cnt + vv) : 0x100000001ull;
+            lq[b] = ok ? __ldg(a.ro + vv + 1) - __ldg(a.ro + vv) : 0;
+          }
+#pragma unroll
+          for (int b = 0; b < kInitU; ++b) {
+            const int64_t len = lq[b];
+            // (rows without entries: the count word is not written, and no item)
+            const bool zero = len > 0 && ((uint32_t)(cq[b] >> 32) == 0u || (uint32_t)cq[b] == 0u);
             const unsigned nsl = __popc(__ballot_sync(kFull, zero && len <= kShortMax));
             const unsigned nwl = __reduce_add_sync(kFull, (zero && len > kShortMax) ? (unsigned)((len + kSeg - 1) / kSeg) : 0u);
             if (lane == 0) {
                 if (nsl) atomicAdd(&stage().nd[0], nsl);
                 if (nwl) atomicAdd(&stage().nd[1], nwl);
             }
+          }
         }
         __syncthreads();
         Stage &st = stage();
@@ -2504,6 +2508,8 @@ static int run_count(gc_graph *g, const RunParams &p, RunResult *r, int jpv) {
     a.n = n;
     a.key = key;
     a.max_rounds = (uint32_t)max_rounds;
+    if (const char *e = std::getenv("GC_MAX_ROUNDS"))  // (experiments: stop after a few rounds)
+        a.max_rounds = (uint32_t)std::min<int64_t>(max_rounds, std::max(0, std::atoi(e)));
     a.sl_cap = (unsigned long long)s.sl_cap;
     a.wl_cap = (unsigned long long)s.wl_cap;
     a.jslot = s.jslot;
