@@ -2121,7 +2121,15 @@ __device__ __forceinline__ void load_tile(const uint32_t *ci, int64_t m, int64_t
     }
 }
 
-__global__ void __launch_bounds__(kWT) k_count_warp(const int64_t *__restrict__ ro, const uint32_t *__restrict__ ci,
+#ifndef GC_CW_PREFETCH
+#define GC_CW_PREFETCH 0  // 1: the next warp tile's column ids loaded before the current one is counted (measured: 1.39 vs 1.23 ms
+                          // without -- 71 vs 55 registers, 24 vs 32 warps per SM)
+#endif
+#ifndef GC_CW_MINB
+#define GC_CW_MINB 1
+#endif
+constexpr bool kCwPrefetch = GC_CW_PREFETCH != 0;
+__global__ void __launch_bounds__(kWT, GC_CW_MINB) k_count_warp(const int64_t *__restrict__ ro, const uint32_t *__restrict__ ci,
                                                     int64_t n, int64_t m, int64_t nch,
                                                     const uint32_t *__restrict__ crow, uint32_t key,
                                                     unsigned long long *cnt, int jp) {
@@ -2138,7 +2146,7 @@ __global__ void __launch_bounds__(kWT) k_count_warp(const int64_t *__restrict__ 
     load_tile(ci, m, w, u);
     for (;;) {
         const int64_t wn = w + nwarps;
-        if (wn < nch) load_tile(ci, m, wn, un);  // next tile's column ids in flight
+        if (kCwPrefetch && wn < nch) load_tile(ci, m, wn, un);  // next tile's column ids in flight
         const int64_t e0 = w * kWE, e1 = min(m, e0 + kWE);
         const int64_t ra = crow[w], rz = crow[w + 1];  // rows touching the tile: [ra, rz]
         const bool last_tile = w == nch - 1;
@@ -2230,8 +2238,12 @@ __global__ void __launch_bounds__(kWT) k_count_warp(const int64_t *__restrict__ 
         }
         if (wn >= nch) break;
         w = wn;
+        if (kCwPrefetch) {
 #pragma unroll
-        for (int q = 0; q < kWQ; ++q) u[q] = un[q];
+            for (int q = 0; q < kWQ; ++q) u[q] = un[q];
+        } else {
+            load_tile(ci, m, w, u);
+        }
     }
 }
 
