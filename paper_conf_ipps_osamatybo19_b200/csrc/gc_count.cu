@@ -2070,7 +2070,10 @@ __global__ void __launch_bounds__(256) k_count_hub(const int64_t *__restrict__ r
 // 64-bit atomic per tile.  Rows without entries are not written: the init
 // phase of the rounds reads their zero degree from the offsets.
 // crow[w] = the row of tile w's first entry (seed-independent, once per graph).
-constexpr int kWQ = 16;             // entries per lane
+#ifndef GC_WQ
+#define GC_WQ 16
+#endif
+constexpr int kWQ = GC_WQ;          // entries per lane
 constexpr int kWE = 32 * kWQ;       // entries per warp tile
 constexpr int kWT = 256;            // threads per block
 constexpr int kTE = kWE;            // (tile granularity of crow / k_count_zero)
