@@ -20,20 +20,27 @@
 // (min wins, Alg.5 L37-42, R9), and a stamp of round k+1 (k+2) never changes a
 // decision of round k+1: the result is the snapshot result (Alg.5 L26, R6)
 // for any interleaving.  Work: the row of every vertex is walked exactly once
-// (when it is coloured) plus one counting pass, so a colouring is O(n + m)
-// with one 8-byte atomic per directed entry; no witness search, no rescans.
+// (when it is coloured) plus one counting pass, so a colouring is O(n + m);
+// the walk issues no atomic for the neighbours on the side of v that was free
+// (all coloured before v's round: their counts are dead), so fewer than one
+// 8-byte atomic per directed entry; no witness search, no rescans.
 //
-// Kernels: k_count (+ k_count_hub for rows > kHubMin) compute hi/lo of every
-// vertex; k_count_persistent then colours round 0 in a dense init phase and
-// runs rounds k = 0, 1, ... over the scheduled lists:
+// Kernels: the counting pass (k_count_zero + k_count_warp: 512-entry warp
+// tiles over the column ids; k_count + k_count_hub for LDF / multi-hash)
+// computes hi/lo of every vertex; k_count_persistent then colours round 0 in
+// a dense init phase and runs rounds k = 0, 1, ... over the scheduled lists:
 //   SL: rows of <= kShortMax entries, one 8-lane group each (4 entries/lane);
-//   WL: longer rows as items of <= kSeg entries, one warp each (8 per lane).
+//   WL: longer rows as items of <= kSeg entries, one warp each.
 // Work units (WL items, groups of 4 SL items) are dealt round-robin over the
 // blocks, so every SM gets an equal share of a round's few thousand units.
 // Items of round k are the slice [end_{k-1}, end_k) of two monotone arrays
-// (each vertex is scheduled once, so the arrays never wrap).  Appends are
-// staged per block in shared memory (one global atomic per list per block per
-// round).
+// (each vertex is scheduled once, so the arrays never wrap).  At a round's
+// end each block takes its slots among the next round's items for the
+// vertices it freed, reserves them with its barrier arrival (one atomic on
+// the round word) and writes them straight to their slots (fresh_flush_direct;
+// the items carry round tags the consumers check).  Max-min rounds k >= 1 are
+// relaxed (no release / acquire): the colours they write are provisional and
+// one pass after the rounds applies the lo-freed-second stamps (DESIGN 7.0).
 
 #include <cstdio>
 #include <cstdlib>
@@ -573,7 +580,8 @@ __device__ __forceinline__ void stage_append(const CArgs &a, bool pred, const It
 // later round reads anything the round writes through a plain load: items
 // carry round tags and are re-read until both halves do, the counts are
 // atomics, and the lo-freed-second stamps and the colours are read only after
-// the rounds, behind one release / acquire barrier (colour_final).
+// the rounds, behind one release / acquire barrier (the final pass of
+// k_count_persistent).
 __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullptr,
                                             unsigned long long t_round = 0, bool relaxed = false) {
     Stage &st = stage();
@@ -1415,7 +1423,7 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
     const int64_t n = a.n;
     // max-min: rounds k >= 1 end with relaxed arrivals; the colours written
     // in the rounds are provisional (max unless the item's side is lo) and
-    // the lo-freed-second stamps are applied after the rounds (colour_final)
+    // the lo-freed-second stamps are applied after the rounds (final pass)
     constexpr bool kRelax = kRelaxedArrive && !JP && !MH;
     // relaxed rounds at run time: max-min always, JP for Luby and Alg.2 (a.jrel:
     // the values a later round reads are read until written, jp_read_once)
