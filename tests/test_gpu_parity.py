@@ -807,3 +807,19 @@ def test_counting_pass_long_isolated_runs():
         dt = time.perf_counter() - t0
     assert k == 1 and st.rounds == 1 and (out.numpy() == 1).all()
     assert dt < 0.5, dt
+
+
+def test_relaxed_rounds_repeated_colourings():
+    """The relaxed rounds (max-min; Luby and Alg.2 through the JP kernel)
+    publish items through round tags and read earlier rounds' single-writer
+    words until written: many colourings with different seeds on ONE handle
+    (item arrays reused across colourings, epoch tags) against the oracle,
+    element by element."""
+    g = G.rmat(16, 16, seed=21)
+    with gcb.Graph(g.n, g.row_offsets, g.col_indices) as h:
+        for seed in range(1, 13):
+            for vname in ("maxmin", "luby", "is_alg2"):
+                out = torch.empty(g.n, dtype=torch.int32)
+                _, _, st = h.color(seed, variant_of(vname), out, stats=True, mode=gcb.MODE_COUNT)
+                assert st.mode_used == gcb.MODE_COUNT
+                assert (out.numpy().view(np.uint32) == oracle_colors(g, seed, vname)).all(), (seed, vname)
