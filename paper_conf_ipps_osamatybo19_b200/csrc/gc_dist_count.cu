@@ -519,7 +519,14 @@ __device__ __forceinline__ void walk_chunks(const DCArgs &a, bool ghost, unsigne
     }
 }
 
-__global__ void __launch_bounds__(256) k_dc_persistent(const __grid_constant__ DPArgs A) {
+#ifndef GC_DC_THREADS
+#define GC_DC_THREADS 256  // threads per block of the partitioned persistent kernel
+#endif
+#ifndef GC_DC_BPS
+#define GC_DC_BPS 3        // its blocks per SM (at most; loopback s22 P=1/2/4/8: 2 -> 21.3/32.6/33.2/36.4 ms,
+                           // 3 -> 20.9/31.7/31.7/33.0, 4 -> 21.6/32.4/31.8/31.7; 512 or 768 threads x 1: slower)
+#endif
+__global__ void __launch_bounds__(GC_DC_THREADS) k_dc_persistent(const __grid_constant__ DPArgs A) {
     const unsigned gsize = gridDim.x / (unsigned)A.nlocal;
     const unsigned lp = blockIdx.x / gsize;
     if (lp >= (unsigned)A.nlocal) return;  // blocks beyond the groups
@@ -946,14 +953,14 @@ int run_dist_persistent(gc_graph *g, const RunParams &p, RunResult *r, int64_t *
     A.nk = reinterpret_cast<int64_t *>(scratch + 32 * kMaxLocal);
     A.nk_cap = nk_cap;
     int per_sm = 0;
-    GC_CUDA_TRY(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_dc_persistent, 256, 0));
-    const int gsize = std::max(1, (std::min(per_sm, 2) * g->sm_count) / nlocal);
+    GC_CUDA_TRY(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_dc_persistent, GC_DC_THREADS, 0));
+    const int gsize = std::max(1, (std::min(per_sm, GC_DC_BPS) * g->sm_count) / nlocal);
     cudaLaunchAttribute attr;
     attr.id = cudaLaunchAttributeCooperative;
     attr.val.cooperative = 1;
     cudaLaunchConfig_t cfg = {};
     cfg.gridDim = dim3((unsigned)(gsize * nlocal));
-    cfg.blockDim = dim3(256);
+    cfg.blockDim = dim3(GC_DC_THREADS);
     cfg.stream = st;
     cfg.attrs = &attr;
     cfg.numAttrs = 1;
