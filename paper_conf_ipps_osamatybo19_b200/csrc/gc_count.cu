@@ -653,9 +653,15 @@ __device__ __forceinline__ void stage_flush(const CArgs &a, int64_t *prs = nullp
 __device__ __forceinline__ void jp_slot_init(const CArgs &a, uint32_t w, int64_t deg);  // (below)
 
 template <bool JP>
-__device__ __forceinline__ void fresh_flush_direct(const CArgs &a, bool relaxed) {
+__device__ __forceinline__ void fresh_flush_direct(const CArgs &a, bool relaxed, int64_t *prs = nullptr,
+                                                   unsigned long long t_round = 0) {
     Stage &st = stage();
     __syncthreads();  // the units are done
+    if (prs && threadIdx.x == 0) {  // PROF (round_stats slots as the staged flush's, tools/freshprof.py)
+        red_max(prs + 7, gtimer() - t_round);
+        red_add(prs + 2, (unsigned long long)st.vis);
+        st.vis = 0;
+    }
     const unsigned nf = min(st.nf, (unsigned)kStF);
     for (unsigned t = threadIdx.x; t < nf; t += blockDim.x) {
         const uint2 f = st.fresh[t];
@@ -673,6 +679,10 @@ __device__ __forceinline__ void fresh_flush_direct(const CArgs &a, bool relaxed)
         st.fmeta[t] = make_uint2((uint32_t)len, pos);
     }
     __syncthreads();
+    if (prs && threadIdx.x == 0) {  // PROF: the fresh vertices' row offsets are in, slots taken
+        red_max(prs + 14, gtimer() - t_round);
+        red_max(prs + 5, gtimer() - t_round);
+    }
     if (threadIdx.x == 0) {
         const unsigned c0 = min(st.n[0], (unsigned)kStS), c1 = min(st.n[1], (unsigned)kStW);
         const unsigned long long t0 = c0 + st.nd[0], t1 = c1 + st.nd[1];
@@ -683,6 +693,10 @@ __device__ __forceinline__ void fresh_flush_direct(const CArgs &a, bool relaxed)
         const unsigned long long rv = relaxed ? atom_add_global(st.rw, rw_add(t0, 0) + rw_add(t1, 1) + kRwArr)
                                               : atom_add_release(st.rw, rw_add(t0, 0) + rw_add(t1, 1) + kRwArr);
         const unsigned long long r0 = rw_field(rv, 0), r1 = rw_field(rv, 1);
+        if (prs) {  // PROF: the reservation (= arrival) came back
+            asm volatile("" ::"l"(rv));
+            red_max(prs + 9, gtimer() - t_round);
+        }
         if (r0 + t0 > kMSL || r1 + t1 > kMWL) flag_error(a, 9, 0, 0);  // a round word field overflowed
         st.base[0] = st.nbase[0] + r0;
         st.base[1] = st.nbase[1] + r1;
@@ -735,6 +749,7 @@ __device__ __forceinline__ void fresh_flush_direct(const CArgs &a, bool relaxed)
         }
     }
     __syncthreads();
+    if (prs && threadIdx.x == 0) red_max(prs + 15, gtimer() - t_round);  // PROF: short items written
     const unsigned nl = min(st.nlong, (unsigned)kLongMax);
     for (unsigned r = threadIdx.x >> 5; r < nl; r += blockDim.x >> 5) {  // a warp per long row
         const Stage::Long L = st.lng[r];
@@ -747,6 +762,10 @@ __device__ __forceinline__ void fresh_flush_direct(const CArgs &a, bool relaxed)
                     ((q == 0 || (JP && a.jpv == 1)) ? L.flags : (L.flags & kLoSide));
             gput(wl + b1 + L.dst + q, si);
         }
+    }
+    if (prs) {  // PROF: every item written
+        __syncthreads();
+        if (threadIdx.x == 0) red_max(prs + 8, gtimer() - t_round);
     }
     // (st.n, st.nd, st.nf are reset at the next round top)
 }
@@ -1675,7 +1694,7 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
                 }
             }
             st.trap = (k & 31u) == 0u ? __ldcg(&a.ctr[cErr]) : 0ull;
-            if (kDirectFlush && !MH && !PROF) {  // (the last round's direct flush is done)
+            if (kDirectFlush && !MH) {  // (the last round's direct flush is done)
                 st.n[0] = st.n[1] = 0;
                 st.nd[0] = st.nd[1] = 0;
                 st.nf = 0;
@@ -1868,8 +1887,8 @@ __global__ void __launch_bounds__((threads_for<JP, MH>()), 1) k_count_persistent
                 }
             }
         }
-        if (kDirectFlush && !MH && !PROF) {
-            fresh_flush_direct<JP>(a, relax);
+        if (kDirectFlush && !MH) {
+            fresh_flush_direct<JP>(a, relax, prs, t_round);
         } else {
             if (!(kEagerFresh && !JP && !MH)) schedule_fresh<JP>(a, prs, t_round);
             stage_flush(a, prs, t_round, relax);
